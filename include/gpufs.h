@@ -1,0 +1,142 @@
+/* gpufs.h — host-side C ABI of libgpufs.so (the B200 GPUfs buffer-cache read path).
+ *
+ * extern "C", plain pointers and sizes only (no torch / CUDA runtime types in
+ * signatures: streams are passed as `void*` holding a cudaStream_t / CUstream,
+ * device buffers as plain pointers). Every call returns 0 or a positive value
+ * on success and -errno on failure.
+ *
+ * Layers (Fig. 2):
+ *   - gfs_init / gfs_shutdown: allocate / free the GPU buffer cache (raw data
+ *     array P:L595-596, pframes P:L597-606, radix-tree nodes P:L612-622, file
+ *     tables) and the per-GPU RPC queue in pinned memory.
+ *   - gfs_daemon / gfs_daemon_stop: the host side of the GPU->CPU RPC
+ *     (P:L675-740): worker threads poll the queue, pread into pinned staging
+ *     and DMA into cache frames, write back dirty ranges, keep a
+ *     close-to-open version table (user-space stand-in for WRAPFS).
+ *   - gfs_run_*: launchers of the kernels built on the device API
+ *     (include/gpufs_device.cuh). They enqueue on `stream` and return without
+ *     synchronising. The daemon must be running while they execute.
+ *
+ * Ownership: the library owns everything it allocates (unless
+ * gfs_config.frame_pool supplies caller-owned device memory for the frames).
+ * Device buffers passed to gfs_run_* are owned by the caller and must stay
+ * valid until the stream reaches the launch. Not thread-safe: call the host
+ * API from one thread per handle.
+ */
+#ifndef GPUFS_H
+#define GPUFS_H
+
+#include <stdint.h>
+#include "gpufs_layout.h"
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct gfs_config {
+  int device;               /* CUDA ordinal */
+  uint64_t cache_bytes;     /* frame pool bytes (paper: 2 GB) */
+  uint32_t page_size;       /* power of two, 4 KiB .. 16 MiB (configurable) */
+  uint32_t ring_slots;      /* RPC queue entries (power of two) */
+  uint32_t daemon_threads;  /* host worker threads (pread + DMA channels) */
+  uint32_t max_files;       /* open+closed file table entries (power of two) */
+  uint32_t max_nodes;       /* radix node pool (0 = auto) */
+  uint32_t max_batch;       /* pages looked up per warp-0 batch, 1..32 */
+  uint32_t flags;           /* GFS_F_* (gpufs_layout.h) */
+  uint32_t pad;
+  uint64_t timeout_ms;      /* device-side wait bound (0 = none) -> -ETIMEDOUT */
+  void* frame_pool;         /* optional caller-owned device memory >= cache_bytes */
+} gfs_config;
+
+typedef struct gfs_handle gfs_handle;
+
+#define GFS_DAEMON_SPAWN 0  /* start worker threads and return */
+#define GFS_DAEMON_RUN 1    /* start workers, block the caller until gfs_daemon_stop */
+
+/* Fill *cfg with defaults (64 KiB pages, 1 GiB cache, 4096 slots, 8 threads). */
+int gfs_config_default(gfs_config* cfg);
+
+/* Allocate the cache and the RPC channel on cfg->device. No kernel may use
+ * the context before this returns. -EINVAL on bad geometry, -ENOMEM on
+ * allocation failure, -ENODEV if CUDA is unavailable. */
+int gfs_init(const gfs_config* cfg, gfs_handle** out);
+
+/* Start the host daemon (mode GFS_DAEMON_SPAWN / GFS_DAEMON_RUN). Uses only
+ * non-blocking streams and never synchronises the device. */
+int gfs_daemon(gfs_handle* h, int mode);
+
+/* Stop the daemon threads (in-flight RPCs are finished first). */
+int gfs_daemon_stop(gfs_handle* h);
+
+/* Free everything. Dirty pages are NOT flushed (gclose != sync). */
+int gfs_shutdown(gfs_handle* h);
+
+/* Device pointer to the gfs_ctx to pass to kernels using gpufs_device.cuh. */
+const gfs_ctx* gfs_device_ctx(gfs_handle* h);
+
+/* Copy the device counters (GFS_C_*, summed over shards) into out[0..n). */
+int gfs_stats(gfs_handle* h, uint64_t* out, int n, int reset);
+
+/* Host daemon counters: out[0..n): rpcs, reads, writes, opens, closes, truncs,
+ * bytes_h2d, bytes_d2h, pread_ns, errors, merges. */
+int gfs_host_stats(gfs_handle* h, uint64_t* out, int n);
+
+/* Geometry: out[0]=page_size out[1]=nframes out[2]=max_files out[3]=max_nodes
+ * out[4]=ring_slots out[5]=daemon_threads out[6]=stream-write-value-64 used. */
+int gfs_info(gfs_handle* h, uint64_t* out, int n);
+
+/* --------------------------------------------------------------------------
+ * Kernel launchers (device-side calls run inside these kernels).
+ * `path` arguments are host NUL-terminated strings; the launcher stages them in
+ * device memory. All d_* pointers are device memory. grid/block: launch shape.
+ * Return 0 once enqueued, -EINVAL on bad arguments, or a CUDA error as -EIO.
+ * ------------------------------------------------------------------------ */
+
+/* Parity harness: each block gopen()s `path` (flags), then issues calls
+ * i = blockIdx.x, blockIdx.x + grid, ... < ncalls:
+ *   mode 0: d_ret[i] = gread(fd, d_off[i], d_len[i], d_dst + d_dstoff[i])
+ *   mode 1: p = gmmap(.., d_len[i], .., fd, d_off[i], &m); copy m bytes to
+ *           d_dst + d_dstoff[i]; gmunmap; d_ret[i] = p ? m : -errno-or-0
+ *   mode 2: like mode 0 but the destination is dynamic shared memory
+ *           (requires d_len[i] <= smem_bytes), copied out to d_dst afterwards
+ * then gclose(). If gopen fails every d_ret[i] of that block gets its error. */
+int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
+                  const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
+                  int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes);
+
+/* Sequential sweep (C2 / K1 shape): block b reads its contiguous
+ * range of [file_off, file_off + total) in `chunk`-byte calls — gread into
+ * d_scratch + b*chunk (use_mmap = 0) or gmmap (use_mmap = 1) — and adds the
+ * position-weighted checksum sum_j w_j*(2j+1) of the bytes read (j = global
+ * 8-byte word index) into *d_sum. Ranges are split in multiples of chunk.
+ * *d_err receives the most negative error seen (0 if none). */
+int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint64_t file_off, uint64_t total,
+                    uint64_t chunk, int use_mmap, uint8_t* d_scratch, uint64_t* d_sum, int64_t* d_err,
+                    uint32_t grid, uint32_t block);
+
+/* Cache-hit read benchmark (K4 shape): block b issues
+ * calls_per_block greads of `chunk` bytes into dynamic shared memory at file
+ * offsets d_off[b*calls_per_block + i] (chunk-aligned), checksumming each
+ * chunk from shared memory into *d_sum. raw != 0 runs the baseline: the same
+ * copies straight from d_raw (the file's bytes already in device memory),
+ * without GPUfs (h may be NULL then). */
+int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
+                     uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
+                     int64_t* d_err, uint32_t grid, uint32_t block);
+
+/* Write harness: each block gopen(path, O_GWRONCE) and issues
+ * d_ret[i] = gwrite(fd, d_off[i], d_len[i], d_src + d_srcoff[i]) for its calls,
+ * then gclose. */
+int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncalls, const uint64_t* d_off,
+                   const uint64_t* d_len, const uint64_t* d_srcoff, const uint8_t* d_src, int64_t* d_ret,
+                   uint32_t grid, uint32_t block);
+
+/* One-block file operations: op 0 = gfsync, 1 = gftruncate(arg), 2 = gfstat_size,
+ * 3 = gopen+gclose only. flags = open flags. *d_ret = result. */
+int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int flags, int op, uint64_t arg,
+                   int64_t* d_ret);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* GPUFS_H */

@@ -1,0 +1,1172 @@
+// gpufs_device.cuh — header-only device library: the GPUfs API called from
+// inside CUDA kernels (sm_100a), block-collectively.
+//
+// API (Table 1; semantics §3.2):
+//
+//   int     gopen (const gfs_ctx*, const char* path, int flags);
+//   int     gclose(const gfs_ctx*, int fd);
+//   int64_t gread (const gfs_ctx*, int fd, uint64_t off, uint64_t len, void* dst);
+//   int64_t gwrite(const gfs_ctx*, int fd, uint64_t off, uint64_t len, const void* src);
+//   int     gfsync(const gfs_ctx*, int fd);
+//   void*   gmmap (const gfs_ctx*, void* addr, uint64_t len, int prot, int flags,
+//                  int fd, uint64_t off, uint64_t* mapped_len);
+//   int     gmunmap(const gfs_ctx*, void* addr, uint64_t len);
+//   int64_t gfstat_size(const gfs_ctx*, int fd);
+//   int     gftruncate(const gfs_ctx*, int fd, uint64_t size);
+//
+// Calling convention (§4): every thread of the threadblock calls
+// the same function with the same arguments at the same point; each call is an
+// implicit barrier and every thread receives the same return value. Negative
+// returns are -errno. `dst`/`src` may point to global or shared memory and are
+// owned by the caller. A gmmap pointer is borrowed until gmunmap.
+//
+// Errors: -EBADF bad/closed fd, gread on O_GWRONCE, gwrite on O_RDONLY;
+// -EINVAL bad flags; -ENOENT/-EACCES from host open; -EMFILE table full;
+// -ENOMEM no evictable frame / node pool exhausted (deadlock guard);
+// -EIO RPC or pread failure; -ENAMETOOLONG path >= GFS_MAX_PATH;
+// -EBUSY gfsync skipped mapped/in-use dirty pages, or conflicting open mode;
+// -ETIMEDOUT the host daemon did not answer within ctx->timeout_ns.
+//
+// Design: per-file radix tree (fanout 256) of u32 frame ids in
+// HBM, looked up lock-free with (uid,page) tag validation; frame
+// state word with refcount + FILLING/EVICTING bits; misses install a frame by
+// CAS, post an RPC on the pinned ring and wait on a device-memory completion
+// word written by the host daemon's stream after its DMA;
+// eviction is a sampled, tiered LRU over 32-frame windows run in the calling
+// thread. Slots are hints: evictors never touch tree nodes, a
+// reader that finds a stale slot installs over it.
+#pragma once
+
+#include <stdint.h>
+#include <errno.h>
+#include "gpufs_layout.h"
+
+
+namespace gfs {
+namespace detail {
+
+// ------------------------------------------------------------------ PTX
+__device__ __forceinline__ uint64_t now_ns() {
+  uint64_t t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+__device__ __forceinline__ uint32_t smid() {
+  uint32_t s;
+  asm volatile("mov.u32 %0, %%smid;" : "=r"(s));
+  return s;
+}
+__device__ __forceinline__ uint32_t ld_acq(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint64_t ld_acq64(const uint64_t* p) {
+  uint64_t v;
+  asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint64_t ld_acq_sys64(const uint64_t* p) {
+  uint64_t v;
+  asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint32_t ld_rlx(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint64_t ld_rlx64(const uint64_t* p) {
+  uint64_t v;
+  asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ void st_rel(uint32_t* p, uint32_t v) {
+  asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+__device__ __forceinline__ void st_rel64(uint64_t* p, uint64_t v) {
+  asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ void st_rel_sys64(uint64_t* p, uint64_t v) {
+  asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ void st_rlx(uint32_t* p, uint32_t v) {
+  asm volatile("st.relaxed.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+__device__ __forceinline__ void st_rlx64(uint64_t* p, uint64_t v) {
+  asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ uint32_t atom_add_acq(uint32_t* p, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.acquire.gpu.global.add.u32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint32_t atom_add_rel(uint32_t* p, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.release.gpu.global.add.u32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint32_t atom_and_rel(uint32_t* p, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.release.gpu.global.and.b32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint32_t atom_or_rel(uint32_t* p, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.release.gpu.global.or.b32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint32_t atom_cas(uint32_t* p, uint32_t cmp, uint32_t val) {
+  uint32_t r;
+  asm volatile("atom.acq_rel.gpu.global.cas.b32 %0, [%1], %2, %3;"
+               : "=r"(r) : "l"(p), "r"(cmp), "r"(val) : "memory");
+  return r;
+}
+__device__ __forceinline__ unsigned long long atom_add64(unsigned long long* p, unsigned long long v) {
+  return atomicAdd(p, v);
+}
+__device__ __forceinline__ void backoff(uint32_t& ns) {
+  __nanosleep(ns);
+  ns = ns < 4096 ? ns * 2 : 4096;
+}
+
+__device__ __forceinline__ void ctr(const gfs_ctx* c, int i, unsigned long long v = 1) {
+  atomicAdd(&c->ctr[(size_t)i * GFS_CTR_SHARDS + (smid() & (GFS_CTR_SHARDS - 1))], v);
+}
+
+__device__ __forceinline__ uint32_t stamp_now() { return (uint32_t)(now_ns() >> 10); }
+
+__device__ __forceinline__ bool timed_out(const gfs_ctx* c, uint64_t t0) {
+  return c->timeout_ns && now_ns() - t0 > c->timeout_ns;
+}
+
+// ------------------------------------------------------------------ thread ids
+__device__ __forceinline__ int block_tid() {
+  return threadIdx.x + blockDim.x * (threadIdx.y + blockDim.y * threadIdx.z);
+}
+__device__ __forceinline__ int block_nthr() { return blockDim.x * blockDim.y * blockDim.z; }
+
+// ------------------------------------------------------------------ scratch
+struct FileSnap {
+  uint32_t fdx, uid, root, height, hfid, oflags;
+  uint64_t size;
+};
+
+struct Scratch {
+  int64_t ret;
+  int64_t aux;
+  void* ptr;
+  FileSnap fs;
+  int32_t frame[GFS_MAX_BATCH];
+  uint32_t installed[GFS_MAX_BATCH];
+  int32_t err;
+  uint32_t busy;
+};
+
+__device__ __forceinline__ Scratch& scratch() {
+  __shared__ Scratch s;
+  return s;
+}
+
+// ------------------------------------------------------------------ RPC client
+// One request on the per-GPU queue: take a ticket, fill the 64-byte
+// slot in pinned host memory, publish seq with st.release.sys (the GPU->CPU
+// fence), then wait for the completion word in HBM that the
+// daemon's stream writes after its DMA. Any thread may call.
+__device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64_t file_off,
+                            uint64_t dev_ptr, uint32_t len, uint32_t flags, uint64_t arg,
+                            const char* path, uint32_t path_len, gfs_rpc_resp* resp_out) {
+  const unsigned long long t = atom_add64(c->ring_tail, 1ull);
+  const uint32_t R = c->ring_slots;
+  const uint32_t slot = (uint32_t)(t % R);
+  const uint64_t t0 = now_ns();
+  uint32_t ns = 32;
+  if (t >= R) {  // slot reuse: its previous client must have released it
+    const uint64_t need = (uint64_t)(t - R + 1);
+    bool waited = false;
+    while (ld_acq64(&c->ack[slot]) != need) {
+      waited = true;
+      backoff(ns);
+      if (timed_out(c, t0)) {
+        ctr(c, GFS_C_TIMEOUT);
+        return -ETIMEDOUT;
+      }
+    }
+    if (waited) ctr(c, GFS_C_RING_WAIT);
+  }
+  volatile gfs_rpc_req* q = c->ring + slot;
+  q->op = op;
+  q->hfid = hfid;
+  q->file_off = file_off;
+  q->dev_ptr = dev_ptr;
+  q->len = len;
+  q->flags = flags;
+  q->arg = arg;
+  q->path_len = path_len;
+  if (path) {
+    volatile char* dp = c->ring_paths + (size_t)slot * GFS_MAX_PATH;
+    for (uint32_t i = 0; i < path_len; ++i) dp[i] = path[i];
+  }
+  st_rel_sys64((uint64_t*)&q->seq, (uint64_t)(t + 1));
+  ctr(c, GFS_C_RPC);
+  const uint32_t want = (uint32_t)(t + 1);
+  uint64_t v;
+  ns = 256;
+  while (((v = ld_acq_sys64(&c->cpl[slot])) >> 32) != want) {
+    backoff(ns);
+    if (timed_out(c, t0)) {
+      ctr(c, GFS_C_TIMEOUT);
+      return -ETIMEDOUT;  // slot is not released: the daemon is gone
+    }
+  }
+  const int32_t res = (int32_t)(uint32_t)(v & 0xFFFFFFFFull);
+  if (resp_out) {
+    volatile gfs_rpc_resp* r = c->resp + slot;
+    resp_out->size = r->size;
+    resp_out->version = r->version;
+    resp_out->ino = r->ino;
+    resp_out->dev = r->dev;
+    resp_out->mtime_ns = r->mtime_ns;
+    resp_out->hfid = r->hfid;
+    resp_out->status = r->status;
+  }
+  st_rel64(&c->ack[slot], (uint64_t)(t + 1));
+  return res;
+}
+
+// ------------------------------------------------------------------ radix nodes
+__device__ __forceinline__ void spin_lock(uint32_t* l) {
+  uint32_t ns = 32;
+  while (atom_cas(l, 0u, 1u) != 0u) backoff(ns);
+}
+__device__ __forceinline__ void spin_unlock(uint32_t* l) { st_rel(l, 0u); }
+
+// Returns a zeroed node index (>= 1; node 0 is reserved as "null"), or 0.
+__device__ uint32_t node_alloc(const gfs_ctx* c) {
+  uint32_t n = 0;
+  spin_lock(c->node_lock);
+  uint32_t top = *(volatile uint32_t*)c->node_free_top;
+  if (top > 0) {
+    n = c->node_free[top - 1];
+    *(volatile uint32_t*)c->node_free_top = top - 1;
+  } else {
+    uint32_t nx = *(volatile uint32_t*)c->node_next;
+    if (nx < c->max_nodes) {
+      n = nx;
+      *(volatile uint32_t*)c->node_next = nx + 1;
+    }
+  }
+  spin_unlock(c->node_lock);
+  if (n) ctr(c, GFS_C_NODES);
+  return n;
+}
+
+__device__ void node_free_one(const gfs_ctx* c, uint32_t n) {
+  uint4* p = (uint4*)(c->nodes + (size_t)n * GFS_FANOUT);
+  for (int i = 0; i < (int)(GFS_FANOUT / 4); ++i) p[i] = make_uint4(0, 0, 0, 0);
+  __threadfence();
+  spin_lock(c->node_lock);
+  uint32_t top = *(volatile uint32_t*)c->node_free_top;
+  c->node_free[top] = n;
+  *(volatile uint32_t*)c->node_free_top = top + 1;
+  spin_unlock(c->node_lock);
+}
+
+// Free every node of a tree (caller guarantees no walker: the file is not open).
+__device__ void tree_free(const gfs_ctx* c, uint32_t root, uint32_t height) {
+  if (!root) return;
+  uint32_t stk_node[GFS_MAX_HEIGHT];
+  uint32_t stk_idx[GFS_MAX_HEIGHT];
+  int sp = 0;
+  stk_node[0] = root;
+  stk_idx[0] = 0;
+  // levels: stack depth d corresponds to node height (height - d)
+  while (sp >= 0) {
+    const uint32_t node = stk_node[sp];
+    const uint32_t h = height - (uint32_t)sp;
+    if (h > 1 && stk_idx[sp] < GFS_FANOUT) {
+      const uint32_t i = stk_idx[sp]++;
+      const uint32_t ch = c->nodes[(size_t)node * GFS_FANOUT + i];
+      if (ch) {
+        ++sp;
+        stk_node[sp] = ch;
+        stk_idx[sp] = 0;
+      }
+      continue;
+    }
+    node_free_one(c, node);
+    --sp;
+  }
+}
+
+// Walk (creating interior nodes if `create`) to the leaf slot of `page`.
+// Interior entries hold child node ids; leaf entries hold frame id + 1.
+// New nodes are zeroed before the publishing CAS.
+__device__ uint32_t* walk(const gfs_ctx* c, uint32_t root, uint32_t height, uint64_t page, bool create,
+                          int* err) {
+  uint32_t node = root;
+  for (int lvl = (int)height - 1; lvl >= 1; --lvl) {
+    const uint32_t idx = (uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & (GFS_FANOUT - 1);
+    uint32_t* sp = c->nodes + (size_t)node * GFS_FANOUT + idx;
+    uint32_t ch = ld_acq(sp);
+    if (!ch) {
+      if (!create) return nullptr;
+      const uint32_t n = node_alloc(c);
+      if (!n) {
+        if (err) *err = -ENOMEM;
+        return nullptr;
+      }
+      __threadfence();
+      const uint32_t prev = atom_cas(sp, 0u, n);
+      if (prev) {
+        node_free_one(c, n);
+        ch = prev;
+      } else {
+        ch = n;
+      }
+    }
+    node = ch;
+  }
+  return c->nodes + (size_t)node * GFS_FANOUT + (uint32_t)(page & (GFS_FANOUT - 1));
+}
+
+__device__ __forceinline__ uint32_t height_for(uint64_t npages) {
+  if (npages <= (1ull << 8)) return 1;
+  if (npages <= (1ull << 16)) return 2;
+  if (npages <= (1ull << 24)) return 3;
+  return 4;
+}
+
+// ------------------------------------------------------------------ frames
+__device__ __forceinline__ uint8_t* frame_ptr(const gfs_ctx* c, uint32_t f) {
+  return c->pool + ((size_t)f << c->page_shift);
+}
+
+__device__ __forceinline__ void frame_init(const gfs_ctx* c, uint32_t f, uint64_t tag, uint32_t fdx) {
+  st_rlx64(&c->f_tag[f], tag);
+  st_rlx(&c->f_file[f], fdx);
+  st_rlx(&c->f_valid[f], 0);
+  st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
+  st_rlx(&c->f_hi[f], 0);
+  st_rlx(&c->f_written[f], 0);
+  st_rlx(&c->f_stamp[f], stamp_now());
+  // EVICTING -> FILLING|1 as an atomic delta: readers that found the frame
+  // through a stale slot may hold transient +1s they are about to undo, so the
+  // state word is never overwritten with a plain store.
+  atom_add_rel(&c->f_state[f], GFS_ST_FILLING + 1u - GFS_ST_EVICTING);
+}
+
+// Write back a frame's dirty range (caller owns it: EVICTING, ref 0).
+__device__ int32_t frame_writeback(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
+  const uint32_t lo = ld_rlx(&c->f_lo[f]);
+  if (lo == GFS_DIRTY_NONE) return 0;
+  const uint32_t hi = ld_rlx(&c->f_hi[f]);
+  const uint32_t wr = ld_rlx(&c->f_written[f]);
+  const uint64_t page = ld_rlx64(&c->f_tag[f]) & 0xFFFFFFFFull;
+  const uint64_t base = page << c->page_shift;
+  const int32_t r = rpc_call(c, GFS_OP_WRITE, hfid, base + lo, (uint64_t)(frame_ptr(c, f) + lo), hi - lo,
+                             wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, nullptr);
+  if (r < 0) return r;
+  st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
+  st_rlx(&c->f_hi[f], 0);
+  st_rlx(&c->f_written[f], 0);
+  ctr(c, GFS_C_WRITEBACK);
+  ctr(c, GFS_C_BYTES_D2H, hi - lo);
+  return 0;
+}
+
+// Tier of a reclaimable frame: 0 orphan/invalid/error,
+// 1 page of a closed file, 2 clean page of an open file, 3 dirty page.
+__device__ __forceinline__ uint32_t frame_tier(const gfs_ctx* c, uint32_t f, uint32_t st) {
+  const uint64_t tag = ld_rlx64(&c->f_tag[f]);
+  if ((st & GFS_ST_ERROR) || tag == GFS_TAG_NONE) return 0;
+  const uint32_t fi = ld_rlx(&c->f_file[f]);
+  if (fi >= c->max_files) return 0;
+  const gfs_file* e = c->files + fi;
+  if (ld_rlx(&e->uid) != (uint32_t)(tag >> 32)) return 0;
+  if (ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) return 3;
+  if ((ld_rlx(&e->sr) >> 24) == GFS_FS_CLOSED) return 1;
+  return 2;
+}
+
+// Allocate a frame for `tag`: never-used frames first, else evict the oldest
+// reclaimable frame of a 32-frame window (sampled LRU, tiered by P:L651-657),
+// writing back a dirty victim first. Runs in the calling thread.
+// Returns the frame in state FILLING|1 with its tag set, or -ENOMEM.
+__device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx) {
+  const uint32_t N = c->nframes;
+  if (ld_rlx(c->fresh_next) < N) {
+    const uint32_t f = atomicAdd(c->fresh_next, 1u);
+    if (f < N) {
+      frame_init(c, f, tag, fdx);
+      return (int)f;
+    }
+  }
+  const uint64_t t0 = now_ns();
+  const uint32_t windows = (N + 31) / 32;
+  uint32_t ns = 64;
+  for (uint32_t round = 0;; ++round) {
+    const uint32_t w = atomicAdd(c->hand, 32u);
+    int best = -1;
+    uint64_t best_key = ~0ull;
+    uint32_t best_st = 0;
+#pragma unroll 4
+    for (uint32_t j = 0; j < 32; ++j) {
+      const uint32_t f = (uint32_t)(((uint64_t)w + j) % N);
+      const uint32_t st = ld_rlx(&c->f_state[f]);
+      if (st & ~GFS_ST_ERROR) continue;  // referenced, filling or being evicted
+      const uint64_t key = ((uint64_t)frame_tier(c, f, st) << 32) | ld_rlx(&c->f_stamp[f]);
+      if (key < best_key) {
+        best_key = key;
+        best = (int)f;
+        best_st = st;
+      }
+    }
+    if (best >= 0 && atom_cas(&c->f_state[best], best_st, GFS_ST_EVICTING) == best_st) {
+      const uint32_t f = (uint32_t)best;
+      if (ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) {
+        const uint32_t fi = ld_rlx(&c->f_file[f]);
+        const int32_t r = frame_writeback(c, f, ld_rlx(&c->files[fi].hfid));
+        if (r < 0) {  // keep the dirty page, try another victim
+          atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+          continue;
+        }
+      }
+      ctr(c, GFS_C_EVICT);
+      frame_init(c, f, tag, fdx);
+      return (int)f;
+    }
+    if (round > 0 && round % windows == 0) {
+      backoff(ns);
+      if (now_ns() - t0 > 2000000000ull) {  // 2 s of full scans: the deadlock guard
+        ctr(c, GFS_C_ENOMEM);
+        return -ENOMEM;
+      }
+    }
+  }
+}
+
+__device__ __forceinline__ void frame_release(const gfs_ctx* c, uint32_t f) {
+  st_rlx(&c->f_stamp[f], stamp_now());
+  atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);  // ref - 1
+}
+
+// Give back a frame we installed but could not publish (lost the CAS race).
+__device__ __forceinline__ void frame_abandon(const gfs_ctx* c, uint32_t f) {
+  st_rel64(&c->f_tag[f], GFS_TAG_NONE);
+  atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+  atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+}
+
+// ------------------------------------------------------------------ page lookup
+// Find page `page` of the snapshot file and take a reference (P:L575-576,
+// P:L616-619). Lock-free: read slot, incref, validate tag == (uid,page)
+// (P:L669-672). Retries once without locking, then takes the file lock on
+// the third attempt. A miss installs a frame by CAS and fills it:
+// READ RPC for O_RDONLY files, or (O_GWRONCE, never fetched) it
+// is returned with *installed = 1 and FILLING still set — the caller's block
+// zero-fills/writes it and clears FILLING.
+__device__ int lookup_page(const gfs_ctx* c, const FileSnap& fs, uint64_t page, uint32_t* installed) {
+  *installed = 0;
+  const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)page;
+  uint32_t* lockp = &c->files[fs.fdx].lock;
+  bool locked = false;
+  if (c->flags & GFS_F_LOCKED_TRAVERSAL) {
+    spin_lock(lockp);
+    locked = true;
+  }
+  int err = 0;
+  uint32_t* slot = walk(c, fs.root, fs.height, page, true, &err);
+  if (!slot) {
+    if (locked) spin_unlock(lockp);
+    return err ? err : -ENOMEM;
+  }
+  const uint64_t t0 = now_ns();
+  int attempt = 0;
+  int result;
+  for (;;) {
+    if (!locked && attempt >= 2) {
+      spin_lock(lockp);
+      locked = true;
+    }
+    if (timed_out(c, t0)) {
+      ctr(c, GFS_C_TIMEOUT);
+      result = -ETIMEDOUT;
+      break;
+    }
+    const uint32_t s = ld_acq(slot);
+    if (s) {
+      const uint32_t f = s - 1;
+      const uint32_t old = atom_add_acq(&c->f_state[f], 1u);
+      uint64_t tag = ld_acq64(&c->f_tag[f]);
+      if (tag == want && !(old & GFS_ST_EVICTING)) {
+        uint32_t st = old;
+        uint32_t ns = 128;
+        while (st & GFS_ST_FILLING) {
+          backoff(ns);
+          st = ld_acq(&c->f_state[f]);
+          if (timed_out(c, t0)) break;
+        }
+        tag = ld_acq64(&c->f_tag[f]);
+        if (tag == want && !(st & (GFS_ST_ERROR | GFS_ST_FILLING))) {
+          ctr(c, GFS_C_HIT);
+          result = (int)f;
+          break;
+        }
+        atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+        if (tag == want && (st & GFS_ST_ERROR) && (old & GFS_ST_FILLING)) {
+          result = -EIO;  // the fill we waited for failed
+          break;
+        }
+        if (st & GFS_ST_FILLING) continue;  // timed out; loop reports it
+      } else {
+        atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+        if (tag == want) {  // being synced or evicted: wait for it to settle
+          uint32_t ns = 128;
+          while (ld_acq64(&c->f_tag[f]) == want && (ld_acq(&c->f_state[f]) & GFS_ST_EVICTING)) {
+            backoff(ns);
+            if (timed_out(c, t0)) break;
+          }
+          ++attempt;
+          ctr(c, GFS_C_RETRY);
+          continue;
+        }
+      }
+      ++attempt;
+      ctr(c, GFS_C_RETRY);
+    }
+    // miss (or stale slot): install a new frame for `want`
+    const int g = alloc_frame(c, want, fs.fdx);
+    if (g < 0) {
+      result = g;
+      break;
+    }
+    if (atom_cas(slot, s, (uint32_t)g + 1u) != s) {
+      frame_abandon(c, (uint32_t)g);
+      ++attempt;
+      ctr(c, GFS_C_RETRY);
+      continue;
+    }
+    if (fs.oflags & GFS_O_GWRONCE) {
+      *installed = 1;
+      ctr(c, GFS_C_ZERO_FILL);
+      result = g;
+      break;
+    }
+    // Fetch min(P, S - pP) bytes from the host into the frame.
+    const uint64_t base = page << c->page_shift;
+    const uint64_t rem = fs.size > base ? fs.size - base : 0;
+    const uint32_t nb = (uint32_t)(rem < c->page_size ? rem : c->page_size);
+    const int32_t r = rpc_call(c, GFS_OP_READ, fs.hfid, base, (uint64_t)frame_ptr(c, (uint32_t)g), nb, 0, 0,
+                               nullptr, 0, nullptr);
+    if (r < 0) {
+      atom_or_rel(&c->f_state[g], GFS_ST_ERROR);
+      atom_and_rel(&c->f_state[g], ~GFS_ST_FILLING);
+      atom_add_rel(&c->f_state[g], 0xFFFFFFFFu);
+      result = r == -ETIMEDOUT ? r : -EIO;
+      break;
+    }
+    st_rlx(&c->f_valid[g], (uint32_t)r);
+    atom_and_rel(&c->f_state[g], ~GFS_ST_FILLING);
+    ctr(c, GFS_C_MISS);
+    ctr(c, GFS_C_RPC_READ);
+    ctr(c, GFS_C_BYTES_H2D, nb);
+    result = g;
+    break;
+  }
+  if (locked) {
+    spin_unlock(lockp);
+    ctr(c, GFS_C_LOCKED);
+  } else {
+    ctr(c, GFS_C_LOCKFREE);
+  }
+  return result;
+}
+
+// ------------------------------------------------------------------ copies
+// Block-cooperative copy of n bytes. Frame reads bypass L1 (ld.global.cg):
+// a frame may have been refilled by DMA since this SM last cached it
+// (P:L693-696). 16-byte vectors with 4 loads in flight per thread when
+// src/dst are co-aligned; 4-byte or byte fallback otherwise.
+__device__ __forceinline__ void block_copy_from_frame(uint8_t* dst, const uint8_t* src, uint64_t n, int tid,
+                                                      int nthr) {
+  if (n == 0) return;
+  if ((((uintptr_t)src ^ (uintptr_t)dst) & 15) == 0) {
+    const uint64_t head = ((16 - ((uintptr_t)src & 15)) & 15) < n ? ((16 - ((uintptr_t)src & 15)) & 15) : n;
+    for (uint64_t i = tid; i < head; i += nthr) dst[i] = __ldcg(src + i);
+    const uint64_t nv = (n - head) >> 4;
+    const int4* s4 = (const int4*)(src + head);
+    int4* d4 = (int4*)(dst + head);
+    uint64_t i = tid;
+    const uint64_t stride = (uint64_t)nthr;
+    for (; i + 3 * stride < nv; i += 4 * stride) {
+      int4 a = __ldcg(s4 + i), b = __ldcg(s4 + i + stride), cc = __ldcg(s4 + i + 2 * stride),
+           d = __ldcg(s4 + i + 3 * stride);
+      d4[i] = a;
+      d4[i + stride] = b;
+      d4[i + 2 * stride] = cc;
+      d4[i + 3 * stride] = d;
+    }
+    for (; i < nv; i += stride) d4[i] = __ldcg(s4 + i);
+    const uint64_t done = head + (nv << 4);
+    for (uint64_t k = done + tid; k < n; k += nthr) dst[k] = __ldcg(src + k);
+  } else if ((((uintptr_t)src ^ (uintptr_t)dst) & 3) == 0) {
+    const uint64_t head = ((4 - ((uintptr_t)src & 3)) & 3) < n ? ((4 - ((uintptr_t)src & 3)) & 3) : n;
+    for (uint64_t i = tid; i < head; i += nthr) dst[i] = __ldcg(src + i);
+    const uint64_t nw = (n - head) >> 2;
+    const uint32_t* s4 = (const uint32_t*)(src + head);
+    uint32_t* d4 = (uint32_t*)(dst + head);
+    for (uint64_t i = tid; i < nw; i += nthr) d4[i] = __ldcg(s4 + i);
+    for (uint64_t k = head + (nw << 2) + tid; k < n; k += nthr) dst[k] = __ldcg(src + k);
+  } else {
+    for (uint64_t i = tid; i < n; i += nthr) dst[i] = __ldcg(src + i);
+  }
+}
+
+// Block-cooperative copy into a frame (gwrite) — plain loads of user data.
+__device__ __forceinline__ void block_copy_to_frame(uint8_t* dst, const uint8_t* src, uint64_t n, int tid, int nthr) {
+  if (n == 0) return;
+  if ((((uintptr_t)src ^ (uintptr_t)dst) & 15) == 0) {
+    const uint64_t head = ((16 - ((uintptr_t)src & 15)) & 15) < n ? ((16 - ((uintptr_t)src & 15)) & 15) : n;
+    for (uint64_t i = tid; i < head; i += nthr) dst[i] = src[i];
+    const uint64_t nv = (n - head) >> 4;
+    const int4* s4 = (const int4*)(src + head);
+    int4* d4 = (int4*)(dst + head);
+    for (uint64_t i = tid; i < nv; i += nthr) d4[i] = s4[i];
+    for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = src[k];
+  } else {
+    for (uint64_t i = tid; i < n; i += nthr) dst[i] = src[i];
+  }
+}
+
+__device__ __forceinline__ void block_zero(uint8_t* dst, uint64_t n, int tid, int nthr) {
+  uint64_t i = tid;
+  const uint64_t head = ((16 - ((uintptr_t)dst & 15)) & 15) < n ? ((16 - ((uintptr_t)dst & 15)) & 15) : n;
+  for (; i < head; i += nthr) dst[i] = 0;
+  const uint64_t nv = (n - head) >> 4;
+  int4* d4 = (int4*)(dst + head);
+  for (uint64_t k = tid; k < nv; k += nthr) d4[k] = make_int4(0, 0, 0, 0);
+  for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = 0;
+}
+
+// ------------------------------------------------------------------ file table
+__device__ __forceinline__ uint64_t path_hash(const char* p, uint32_t n) {
+  uint64_t h = 1469598103934665603ull;
+  for (uint32_t i = 0; i < n; ++i) h = (h ^ (uint8_t)p[i]) * 1099511628211ull;
+  return h;
+}
+
+__device__ __forceinline__ bool snap_fd(const gfs_ctx* c, int fd, FileSnap* s) {
+  if (fd < 0 || (uint32_t)fd >= c->max_files) return false;
+  const gfs_file* e = c->files + fd;
+  const uint32_t sr = ld_acq(&e->sr);
+  if ((sr >> 24) != GFS_FS_OPEN || (sr & 0xFFFFFF) == 0) return false;
+  // relaxed (L2) loads: an entry can be re-incarnated by another SM while
+  // this SM still holds an L1 line of it from earlier in the launch
+  s->fdx = (uint32_t)fd;
+  s->uid = ld_rlx(&e->uid);
+  s->root = ld_rlx(&e->root);
+  s->height = ld_rlx(&e->height);
+  s->hfid = ld_rlx(&e->hfid);
+  s->oflags = ld_rlx(&e->oflags);
+  s->size = ld_rlx64((const uint64_t*)&e->size);
+  return true;
+}
+
+// Write back every dirty, unreferenced page of the snapshot file in pages
+// [pb, pe), strided over the calling threads. Returns 0, -EBUSY (a dirty page
+// was mapped or in use, Tab.1), or a negative RPC error.
+__device__ int sync_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uint64_t pe, int tid, int nthr) {
+  int rc = 0;
+  for (uint64_t p = pb + tid; p < pe; p += nthr) {
+    uint32_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
+    if (!slot) continue;
+    const uint32_t s = ld_acq(slot);
+    if (!s) continue;
+    const uint32_t f = s - 1;
+    const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
+    if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) continue;
+    if (atom_cas(&c->f_state[f], 0u, GFS_ST_EVICTING) != 0u) {
+      if (ld_acq64(&c->f_tag[f]) == want && ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE && rc == 0) rc = -EBUSY;
+      continue;
+    }
+    if (ld_acq64(&c->f_tag[f]) == want) {
+      const int32_t r = frame_writeback(c, f, fs.hfid);
+      if (r < 0) rc = r;
+    }
+    atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+  }
+  return rc;
+}
+
+// Drop cached pages [pb, pe) of the snapshot file (gftruncate / invalidation).
+__device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uint64_t pe, int tid, int nthr) {
+  int rc = 0;
+  for (uint64_t p = pb + tid; p < pe; p += nthr) {
+    uint32_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
+    if (!slot) continue;
+    const uint32_t s = ld_acq(slot);
+    if (!s) continue;
+    const uint32_t f = s - 1;
+    const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
+    if (ld_acq64(&c->f_tag[f]) != want) continue;
+    if (atom_cas(&c->f_state[f], 0u, GFS_ST_EVICTING) != 0u) {
+      rc = -EBUSY;
+      continue;
+    }
+    if (ld_acq64(&c->f_tag[f]) == want) {
+      st_rlx64(&c->f_tag[f], GFS_TAG_NONE);
+      st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
+      st_rlx(&c->f_hi[f], 0);
+      st_rlx(&c->f_written[f], 0);
+    }
+    atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+  }
+  return rc;
+}
+
+__device__ __forceinline__ bool same_path(const gfs_ctx* c, const gfs_file* e, uint32_t fdx, const char* path,
+                                          uint32_t n, uint64_t h) {
+  if (ld_rlx64(&e->path_hash) != h || ld_rlx(&e->path_len) != n) return false;
+  const volatile char* sp = c->paths + (size_t)fdx * GFS_MAX_PATH;
+  for (uint32_t i = 0; i < n; ++i)
+    if (sp[i] != path[i]) return false;
+  return true;
+}
+
+// Open RPC + install of a fresh incarnation. `e` is held in OPENING/REOPENING.
+__device__ int open_rpc_fill(const gfs_ctx* c, gfs_file* e, uint32_t fdx, uint32_t flags, uint32_t old_hfid_plus1,
+                             gfs_rpc_resp* rs) {
+  const char* sp = c->paths + (size_t)fdx * GFS_MAX_PATH;
+  const int32_t r = rpc_call(c, GFS_OP_OPEN, 0, 0, 0, 0, flags, old_hfid_plus1, sp, e->path_len, rs);
+  ctr(c, GFS_C_RPC_OPEN);
+  if (r < 0) return r;
+  if (rs->status < 0) return rs->status;
+  return 0;
+}
+
+__device__ int new_incarnation(const gfs_ctx* c, gfs_file* e, uint32_t flags, const gfs_rpc_resp& rs) {
+  const uint32_t root = node_alloc(c);
+  if (!root) return -ENOMEM;
+  const uint64_t P = c->page_size;
+  const uint64_t npages = ((uint64_t)rs.size + P - 1) >> c->page_shift;
+  e->root = root;
+  e->height = (flags & GFS_O_GWRONCE) ? GFS_MAX_HEIGHT : height_for(npages);
+  e->uid = atomicAdd(c->uid_next, 1u);
+  e->hfid = rs.hfid;
+  e->size = (uint64_t)rs.size;
+  e->version = rs.version;
+  e->ino = rs.ino;
+  e->dev = rs.dev;
+  e->mtime_ns = rs.mtime_ns;
+  e->oflags = flags;
+  return 0;
+}
+
+// gopen body, run by one thread.
+__device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
+  if (flags != (int)GFS_O_RDONLY && flags != (int)GFS_O_GWRONCE) return -EINVAL;
+  uint32_t n = 0;
+  while (n < GFS_MAX_PATH && path[n]) ++n;
+  if (n == 0) return -ENOENT;
+  if (n >= GFS_MAX_PATH) return -ENAMETOOLONG;
+  const uint64_t h = path_hash(path, n);
+  const uint32_t mask = c->max_files - 1;
+  uint32_t i = (uint32_t)h & mask;
+  uint32_t probes = 0;
+  const uint64_t t0 = now_ns();
+  uint32_t ns = 64;
+  for (;;) {
+    if (probes > c->max_files) return -EMFILE;
+    gfs_file* e = c->files + i;
+    const uint32_t sr = ld_acq(&e->sr);
+    const uint32_t st = sr >> 24;
+    if (st == GFS_FS_FREE) {
+      if (atom_cas(&e->sr, 0u, (GFS_FS_CLAIM << 24) | 1u) != 0u) continue;
+      char* sp = c->paths + (size_t)i * GFS_MAX_PATH;
+      for (uint32_t k = 0; k < n; ++k) sp[k] = path[k];
+      sp[n] = 0;
+      e->path_len = n;
+      e->path_hash = h;
+      e->lock = 0;
+      e->err = 0;
+      st_rel(&e->sr, (GFS_FS_OPENING << 24) | 1u);
+      gfs_rpc_resp rs;
+      int r = open_rpc_fill(c, e, i, (uint32_t)flags, 0, &rs);
+      if (r == 0) r = new_incarnation(c, e, (uint32_t)flags, rs);
+      if (r < 0) {
+        e->err = r;
+        st_rel(&e->sr, GFS_FS_DEAD << 24);  // tombstone; a later gopen retries further along
+        return r;
+      }
+      st_rel(&e->sr, (GFS_FS_OPEN << 24) | 1u);
+      return (int)i;
+    }
+    if (st == GFS_FS_CLAIM) {  // being inserted: wait for its path
+      backoff(ns);
+      if (timed_out(c, t0)) return -ETIMEDOUT;
+      continue;
+    }
+    if (!same_path(c, e, i, path, n, h)) {
+      i = (i + 1) & mask;
+      ++probes;
+      continue;
+    }
+    if (st == GFS_FS_DEAD) {
+      i = (i + 1) & mask;
+      ++probes;
+      continue;
+    }
+    if (st == GFS_FS_OPENING || st == GFS_FS_REOPENING) {
+      backoff(ns);
+      if (timed_out(c, t0)) return -ETIMEDOUT;
+      continue;
+    }
+    if (st == GFS_FS_OPEN) {
+      if (e->oflags != (uint32_t)flags) return -EBUSY;  // one writer at a time
+      if (atom_cas(&e->sr, sr, sr + 1) == sr) {
+        ctr(c, GFS_C_OPEN_FAST);  // no CPU communication
+        return (int)i;
+      }
+      continue;
+    }
+    if (st == GFS_FS_CLOSED) {
+      if (atom_cas(&e->sr, sr, (GFS_FS_REOPENING << 24) | 1u) != sr) continue;
+      // Closed-file cache: re-open validates against the host (lazy
+      // invalidation). O_GWRONCE or a mode change always starts
+      // a fresh incarnation (pristine copy = zeros).
+      FileSnap old;
+      old.fdx = i; old.uid = e->uid; old.root = e->root; old.height = e->height;
+      old.hfid = e->hfid; old.oflags = e->oflags; old.size = e->size;
+      if (old.oflags & GFS_O_GWRONCE) {  // never lose written data: sync before dropping
+        const uint64_t np = (old.size + c->page_size - 1) >> c->page_shift;
+        int r = sync_pages(c, old, 0, np, 0, 1);
+        if (r < 0 && r != -EBUSY) {
+          st_rel(&e->sr, GFS_FS_CLOSED << 24);
+          return r;
+        }
+      }
+      gfs_rpc_resp rs;
+      int r = open_rpc_fill(c, e, i, (uint32_t)flags, old.hfid + 1u, &rs);
+      if (r < 0) {
+        st_rel(&e->sr, GFS_FS_CLOSED << 24);
+        return r;
+      }
+      const bool same = (uint32_t)flags == GFS_O_RDONLY && old.oflags == GFS_O_RDONLY &&
+                        rs.version == e->version && (uint64_t)rs.size == e->size && rs.ino == e->ino &&
+                        rs.dev == e->dev && rs.mtime_ns == e->mtime_ns;
+      if (same) {
+        e->hfid = rs.hfid;
+        ctr(c, GFS_C_REOPEN_VALID);
+      } else {
+        tree_free(c, old.root, old.height);  // old frames become orphans (tier 0)
+        r = new_incarnation(c, e, (uint32_t)flags, rs);
+        ctr(c, GFS_C_INVALIDATE);
+        if (r < 0) {
+          e->err = r;
+          st_rel(&e->sr, GFS_FS_DEAD << 24);
+          return r;
+        }
+      }
+      st_rel(&e->sr, (GFS_FS_OPEN << 24) | 1u);
+      return (int)i;
+    }
+    i = (i + 1) & mask;  // unknown state: skip
+    ++probes;
+  }
+}
+
+__device__ int close_leader(const gfs_ctx* c, int fd) {
+  if (fd < 0 || (uint32_t)fd >= c->max_files) return -EBADF;
+  gfs_file* e = c->files + fd;
+  for (;;) {
+    const uint32_t sr = ld_acq(&e->sr);
+    if ((sr >> 24) != GFS_FS_OPEN || (sr & 0xFFFFFF) == 0) return -EBADF;
+    const uint32_t nsr = (sr & 0xFFFFFF) == 1 ? (GFS_FS_CLOSED << 24) : sr - 1;
+    if (atom_cas(&e->sr, sr, nsr) == sr) return 0;  // no write-back
+  }
+}
+
+}  // namespace detail
+
+// ===================================================================== API
+using detail::Scratch;
+
+// gopen: returns an fd shared by all openers of the path on this GPU.
+__device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
+  Scratch& sc = detail::scratch();
+  __syncthreads();
+  if (detail::block_tid() == 0) sc.ret = detail::open_leader(c, path, flags);
+  __syncthreads();
+  return (int)sc.ret;
+}
+
+// gclose: drops this block's reference; never writes back.
+__device__ inline int gclose(const gfs_ctx* c, int fd) {
+  Scratch& sc = detail::scratch();
+  __syncthreads();
+  if (detail::block_tid() == 0) sc.ret = detail::close_leader(c, fd);
+  __syncthreads();
+  return (int)sc.ret;
+}
+
+__device__ inline int64_t gfstat_size(const gfs_ctx* c, int fd) {
+  Scratch& sc = detail::scratch();
+  __syncthreads();
+  if (detail::block_tid() == 0) {
+    detail::FileSnap s;
+    sc.ret = detail::snap_fd(c, fd, &s) ? (int64_t)s.size : -EBADF;
+  }
+  __syncthreads();
+  return sc.ret;
+}
+
+// gread: pread semantics; returns min(len, S-off) bytes, 0 at/after EOF.
+__device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+  using namespace detail;
+  Scratch& sc = scratch();
+  const int tid = block_tid(), nthr = block_nthr();
+  __syncthreads();
+  if (tid == 0) {
+    FileSnap s;
+    if (!snap_fd(c, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
+      sc.ret = -EBADF;
+    } else {
+      sc.fs = s;
+      sc.ret = off >= s.size ? 0 : (int64_t)(len < s.size - off ? len : s.size - off);
+      ctr(c, GFS_C_GREAD_CALLS);
+      if (sc.ret > 0) ctr(c, GFS_C_GREAD_BYTES, (unsigned long long)sc.ret);
+    }
+  }
+  __syncthreads();
+  const int64_t n = sc.ret;
+  if (n <= 0) return n;
+  const FileSnap fs = sc.fs;
+  const uint32_t shift = c->page_shift;
+  const uint64_t P = c->page_size;
+  const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
+  const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
+  for (uint64_t pb = p0; pb <= p1; pb += B) {
+    const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
+    if (tid < (int)cnt) {
+      uint32_t inst;
+      sc.frame[tid] = lookup_page(c, fs, pb + tid, &inst);
+    }
+    __syncthreads();
+    int err = 0;
+    for (uint32_t i = 0; i < cnt; ++i)
+      if (sc.frame[i] < 0) err = sc.frame[i];
+    if (!err) {
+      for (uint32_t i = 0; i < cnt; ++i) {
+        const uint64_t p = pb + i;
+        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+        block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+                              e - s, tid, nthr);
+      }
+    }
+    __syncthreads();
+    if (tid < (int)cnt && sc.frame[tid] >= 0) frame_release(c, (uint32_t)sc.frame[tid]);
+    if (err) return err;
+  }
+  return n;
+}
+
+// gwrite: pwrite semantics on an O_GWRONCE file.
+// New pages are zero-filled (never fetched); the dirty range and written byte
+// count are kept per frame; a fence makes the data visible to write-back DMA
+// (P:L577-582).
+__device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, const void* src) {
+  using namespace detail;
+  Scratch& sc = scratch();
+  const int tid = block_tid(), nthr = block_nthr();
+  __syncthreads();
+  if (tid == 0) {
+    FileSnap s;
+    if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_GWRONCE)) {
+      sc.ret = -EBADF;
+    } else if (off + len < off || ((off + len) >> c->page_shift) >= (1ull << 32)) {
+      sc.ret = -EINVAL;
+    } else {
+      sc.fs = s;
+      sc.ret = (int64_t)len;
+      ctr(c, GFS_C_GWRITE_CALLS);
+    }
+  }
+  __syncthreads();
+  const int64_t n = sc.ret;
+  if (n <= 0) return n;
+  const FileSnap fs = sc.fs;
+  const uint32_t shift = c->page_shift;
+  const uint64_t P = c->page_size;
+  const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
+  const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
+  for (uint64_t pb = p0; pb <= p1; pb += B) {
+    const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
+    if (tid < (int)cnt) {
+      uint32_t inst = 0;
+      sc.frame[tid] = lookup_page(c, fs, pb + tid, &inst);
+      sc.installed[tid] = inst;
+    }
+    __syncthreads();
+    int err = 0;
+    for (uint32_t i = 0; i < cnt; ++i)
+      if (sc.frame[i] < 0) err = sc.frame[i];
+    if (!err) {
+      for (uint32_t i = 0; i < cnt; ++i) {
+        const uint64_t p = pb + i;
+        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+        uint8_t* fp = frame_ptr(c, (uint32_t)sc.frame[i]);
+        if (sc.installed[i]) {  // pristine copy is zeros
+          block_zero(fp, s, tid, nthr);
+          block_zero(fp + e, P - e, tid, nthr);
+        }
+        block_copy_to_frame(fp + s, (const uint8_t*)src + ((p << shift) + s - off), e - s, tid, nthr);
+      }
+      __threadfence();
+    }
+    __syncthreads();
+    if (tid < (int)cnt && sc.frame[tid] >= 0) {
+      const uint32_t f = (uint32_t)sc.frame[tid];
+      if (!err) {
+        const uint64_t p = pb + tid;
+        const uint32_t s = (uint32_t)(p == p0 ? (off & (P - 1)) : 0);
+        const uint32_t e = (uint32_t)(p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P);
+        atomicMin(&c->f_lo[f], s);
+        atomicMax(&c->f_hi[f], e);
+        atomicAdd(&c->f_written[f], e - s);
+      }
+      if (sc.installed[tid]) atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+      frame_release(c, f);
+    }
+    if (err) return err;
+  }
+  if (tid == 0) atomicMax((unsigned long long*)&c->files[fd].size, (unsigned long long)(off + (uint64_t)n));
+  __syncthreads();
+  return n;
+}
+
+// gfsync: synchronously write back all dirty pages of the file that are not
+// mapped or in use (Tab.1); on success the data is in the host page
+// cache. Returns -EBUSY if busy dirty pages were skipped.
+__device__ inline int gfsync(const gfs_ctx* c, int fd) {
+  using namespace detail;
+  Scratch& sc = scratch();
+  const int tid = block_tid(), nthr = block_nthr();
+  __syncthreads();
+  if (tid == 0) {
+    FileSnap s;
+    if (!snap_fd(c, fd, &s)) {
+      sc.ret = -EBADF;
+    } else {
+      sc.fs = s;
+      sc.ret = 0;
+      sc.err = 0;
+    }
+  }
+  __syncthreads();
+  if (sc.ret < 0) return (int)sc.ret;
+  const FileSnap fs = sc.fs;
+  if (fs.oflags & GFS_O_GWRONCE) {
+    const uint64_t np = (fs.size + c->page_size - 1) >> c->page_shift;
+    const int r = sync_pages(c, fs, 0, np, tid, nthr);
+    if (r < 0) atomicMin(&sc.err, r);  // any error: -EIO etc. are < -EBUSY
+  }
+  __syncthreads();
+  return sc.err;
+}
+
+// gmmap: map a prefix of at most one cache page;
+// returns a pointer straight into the frame, NULL at/after EOF
+// or on error. *mapped_len = min(len, P - off%P, S - off). MAP_FIXED (addr) is
+// ignored; prot is not enforced.
+__device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int prot, int flags, int fd, uint64_t off,
+                              uint64_t* mapped_len) {
+  using namespace detail;
+  (void)addr;
+  (void)prot;
+  (void)flags;
+  Scratch& sc = scratch();
+  const int tid = block_tid();
+  __syncthreads();
+  if (tid == 0) {
+    FileSnap s;
+    sc.ptr = nullptr;
+    sc.aux = 0;
+    if (!snap_fd(c, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
+      sc.aux = -EBADF;
+    } else if (off < s.size && len > 0) {
+      uint32_t inst;
+      const int f = lookup_page(c, s, off >> c->page_shift, &inst);
+      if (f < 0) {
+        sc.aux = f;
+      } else {
+        const uint64_t in = off & (c->page_size - 1);
+        uint64_t m = c->page_size - in;
+        if (len < m) m = len;
+        if (s.size - off < m) m = s.size - off;
+        sc.ptr = frame_ptr(c, (uint32_t)f) + in;
+        sc.aux = (int64_t)m;
+      }
+    }
+  }
+  __syncthreads();
+  if (mapped_len) *mapped_len = sc.aux > 0 ? (uint64_t)sc.aux : 0;
+  return sc.ptr;
+}
+
+// gmunmap: release the page reference; the frame is found from the pointer
+// (i-th pframe <-> i-th page).
+__device__ inline int gmunmap(const gfs_ctx* c, void* addr, uint64_t len) {
+  using namespace detail;
+  (void)len;
+  Scratch& sc = scratch();
+  __syncthreads();
+  if (block_tid() == 0) {
+    const uint8_t* p = (const uint8_t*)addr;
+    if (p < c->pool || p >= c->pool + ((size_t)c->nframes << c->page_shift)) {
+      sc.ret = -EINVAL;
+    } else {
+      frame_release(c, (uint32_t)((size_t)(p - c->pool) >> c->page_shift));
+      sc.ret = 0;
+    }
+  }
+  __syncthreads();
+  return (int)sc.ret;
+}
+
+// gftruncate: host ftruncate and reclaim cached pages beyond the new size
+// (Tab.1; used by the mat-vec output).
+__device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
+  using namespace detail;
+  Scratch& sc = scratch();
+  const int tid = block_tid(), nthr = block_nthr();
+  __syncthreads();
+  if (tid == 0) {
+    FileSnap s;
+    if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_GWRONCE)) {
+      sc.ret = -EBADF;
+    } else {
+      sc.fs = s;
+      sc.err = 0;
+      const int32_t r = rpc_call(c, GFS_OP_TRUNC, s.hfid, 0, 0, 0, 0, size, nullptr, 0, nullptr);
+      sc.ret = r < 0 ? r : 0;
+      if (r >= 0) st_rlx64((uint64_t*)&c->files[fd].size, size);
+    }
+  }
+  __syncthreads();
+  if (sc.ret < 0) return (int)sc.ret;
+  const FileSnap fs = sc.fs;
+  const uint64_t P = c->page_size;
+  const uint64_t first = (size + P - 1) >> c->page_shift;
+  const uint64_t np = (fs.size + P - 1) >> c->page_shift;
+  if (np > first) {
+    const int r = drop_pages(c, fs, first, np, tid, nthr);
+    if (r < 0) atomicMin(&sc.err, r);
+  }
+  __syncthreads();
+  return sc.err;
+}
+
+}  // namespace gfs

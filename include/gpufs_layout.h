@@ -1,0 +1,189 @@
+/* gpufs_layout.h — memory layout shared by the host runtime (libgpufs.so) and
+ * the header-only device library (gpufs_device.cuh). Plain C, no CUDA types.
+ *
+ * Everything here lives in one of three places (Fig. 2, §4):
+ *   HBM (device memory)        — frame pool ("raw data array"),
+ *                                per-frame metadata ("pframes"),
+ *                                radix-tree node pool, open/closed
+ *                                file table, RPC completion words;
+ *   pinned, mapped host memory — the per-GPU RPC request queue;
+ *   host only                  — daemon state (fd table, staging, streams).
+ */
+#ifndef GPUFS_LAYOUT_H
+#define GPUFS_LAYOUT_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+/* ---- limits ---------------------------------------------------------- */
+#define GFS_MAX_PATH 1024u     /* bytes incl. NUL; longer paths -> -ENAMETOOLONG */
+#define GFS_FANOUT_SHIFT 8u    /* radix tree fanout 256 */
+#define GFS_FANOUT (1u << GFS_FANOUT_SHIFT)
+#define GFS_MAX_HEIGHT 4u      /* 256^4 = 2^32 pages per file */
+#define GFS_MAX_BATCH 32u      /* pages looked up per warp-0 batch (one per lane) */
+#define GFS_CTR_SHARDS 32      /* counters are sharded by SM id to avoid a hot address */
+
+/* ---- open flags ------------------------------------------ */
+#define GFS_O_RDONLY 0u
+#define GFS_O_GWRONCE 1u       /* write-once, pages never fetched, pristine = zeros */
+
+/* ---- config flags ------------------------------------------------------ */
+#define GFS_F_LOCKED_TRAVERSAL 1u /* K5 ablation: every lookup takes the file lock */
+#define GFS_F_NO_DMA_COMPLETION 2u /* fallback: completion via memcpy instead of stream write-value */
+
+/* ---- frame state word (pframe "state") ---------------------------------
+ * bits 0..23  reference count (gread/gwrite copies and gmmap mappings)
+ * bit  24     FILLING  — frame installed, contents not yet valid
+ * bit  25     EVICTING — claimed by eviction / gfsync / truncate (ref was 0)
+ * bit  26     ERROR    — fill failed; readers get -EIO
+ */
+#define GFS_ST_REF_MASK 0x00FFFFFFu
+#define GFS_ST_FILLING (1u << 24)
+#define GFS_ST_EVICTING (1u << 25)
+#define GFS_ST_ERROR (1u << 26)
+#define GFS_TAG_NONE 0xFFFFFFFFFFFFFFFFull /* tag = (uid << 32) | page index */
+#define GFS_DIRTY_NONE 0xFFFFFFFFu
+
+/* ---- file table entry states (high byte of `sr`; low 24 bits = refcount) */
+#define GFS_FS_FREE 0u
+#define GFS_FS_CLAIM 1u
+#define GFS_FS_OPENING 2u
+#define GFS_FS_OPEN 3u
+#define GFS_FS_CLOSED 4u
+#define GFS_FS_REOPENING 5u
+#define GFS_FS_DEAD 6u
+
+typedef struct gfs_file {
+  uint32_t sr;        /* (state << 24) | threadblock refcount */
+  uint32_t uid;       /* cache incarnation id, never reused */
+  uint32_t hfid;      /* daemon's host file id */
+  uint32_t root;      /* radix root node index */
+  uint64_t size;      /* size at first gopen / max written end */
+  uint64_t version;   /* close-to-open version seen at (re)open */
+  uint64_t ino, dev;
+  int64_t mtime_ns;
+  uint64_t path_hash;
+  uint32_t path_len;
+  uint32_t height;
+  uint32_t oflags;
+  uint32_t lock;      /* file spinlock for locked traversal */
+  int32_t err;
+  uint32_t pad;
+} gfs_file;
+
+/* ---- RPC (§4.3) -------------------------------------------- */
+#define GFS_OP_NOP 0u
+#define GFS_OP_OPEN 1u     /* path -> hfid, size, version, ino, dev, mtime */
+#define GFS_OP_READ 2u     /* pread(hfid, len, off) -> DMA to dev_ptr */
+#define GFS_OP_WRITE 3u    /* DMA from dev_ptr -> pwrite(hfid, len, off), version++ */
+#define GFS_OP_CLOSE 4u    /* close(hfid) */
+#define GFS_OP_TRUNC 5u    /* ftruncate(hfid, arg) */
+
+#define GFS_WF_FULL 1u     /* WRITE: every byte of [off,off+len) was written (no merge) */
+
+typedef struct gfs_rpc_req { /* one 64-byte ring slot in pinned host memory */
+  uint32_t op;
+  uint32_t hfid;
+  uint64_t file_off;
+  uint64_t dev_ptr;
+  uint32_t len;
+  uint32_t flags;
+  uint64_t arg;
+  uint32_t path_len;
+  uint32_t pad0;
+  uint64_t pad1;
+  uint64_t seq;      /* = ticket + 1; written LAST with st.release.sys */
+} gfs_rpc_req;
+
+typedef struct gfs_rpc_resp { /* OPEN reply, host-written before completion */
+  int64_t size;
+  uint64_t version;
+  uint64_t ino, dev;
+  int64_t mtime_ns;
+  uint32_t hfid;
+  int32_t status;
+  uint64_t pad[2];
+} gfs_rpc_resp;
+
+/* completion word (device memory): ((ticket + 1) << 32) | (uint32_t)result */
+
+/* ---- counters (Table 2 analogue + RPC accounting) --------------------- */
+enum {
+  GFS_C_HIT = 0,        /* page found valid, lock-free */
+  GFS_C_MISS,           /* page installed and fetched from host */
+  GFS_C_ZERO_FILL,      /* O_GWRONCE page installed zero-filled */
+  GFS_C_LOCKFREE,       /* lookups that succeeded without the lock */
+  GFS_C_LOCKED,         /* lookups that took the file lock (incl. retries) */
+  GFS_C_RETRY,          /* optimistic validation failures */
+  GFS_C_EVICT,          /* frames reclaimed */
+  GFS_C_WRITEBACK,      /* dirty ranges written back */
+  GFS_C_RPC,            /* RPCs posted */
+  GFS_C_RPC_OPEN,
+  GFS_C_RPC_READ,
+  GFS_C_RPC_WRITE,
+  GFS_C_BYTES_H2D,
+  GFS_C_BYTES_D2H,
+  GFS_C_OPEN_FAST,      /* gopen served without RPC */
+  GFS_C_REOPEN_VALID,   /* closed-file cache revalidated and kept */
+  GFS_C_INVALIDATE,     /* closed-file cache dropped on re-open */
+  GFS_C_ENOMEM,
+  GFS_C_TIMEOUT,
+  GFS_C_GREAD_CALLS,
+  GFS_C_GREAD_BYTES,
+  GFS_C_GWRITE_CALLS,
+  GFS_C_NODES,          /* radix nodes allocated */
+  GFS_C_RING_WAIT,      /* ring slot was busy on post */
+  GFS_C_NCOUNTERS
+};
+
+/* ---- the device context (lives in HBM; kernels receive a pointer) ------ */
+typedef struct gfs_ctx {
+  uint64_t page_size;
+  uint32_t page_shift;
+  uint32_t nframes;
+  uint8_t* pool;
+  /* pframes, SoA */
+  uint32_t* f_state;
+  uint64_t* f_tag;
+  uint32_t* f_file;
+  uint32_t* f_valid;
+  uint32_t* f_lo;
+  uint32_t* f_hi;
+  uint32_t* f_written;
+  uint32_t* f_stamp;
+  uint32_t* fresh_next;
+  uint32_t* hand;
+  /* radix node pool */
+  uint32_t* nodes;
+  uint32_t max_nodes;
+  uint32_t max_files; /* power of two */
+  uint32_t* node_next;
+  uint32_t* node_free;
+  uint32_t* node_free_top;
+  uint32_t* node_lock;
+  /* file table */
+  gfs_file* files;
+  char* paths;
+  uint32_t* uid_next;
+  uint32_t ring_slots;
+  /* RPC */
+  gfs_rpc_req* ring;   /* device-mapped pointer to pinned host ring */
+  gfs_rpc_resp* resp;  /* device-mapped pointer to pinned host responses */
+  char* ring_paths;    /* device-mapped, ring_slots * GFS_MAX_PATH */
+  uint64_t* cpl;       /* device memory completion words */
+  uint64_t* ack;       /* device memory: slot released by its client */
+  unsigned long long* ring_tail;
+  /* config */
+  uint32_t flags;
+  uint32_t max_batch;
+  uint64_t timeout_ns;
+  unsigned long long* ctr;
+} gfs_ctx;
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* GPUFS_LAYOUT_H */

@@ -1,0 +1,168 @@
+"""paper_conf_asplos_silbersteinfkw13_b200 — B200-native GPUfs buffer-cache read path.
+
+Thin Python binding over ``libgpufs.so`` (include/gpufs.h): argument
+marshalling only. Every step of the path (gopen, radix lookup, miss RPC,
+eviction, hit copy, gwrite/gfsync, the consumer kernels) runs in the CUDA
+library and its host daemon. PyTorch is used only for device memory and
+streams. There is no CPU fallback: if the library is missing or no GPU is
+present, the calls raise.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+_PKG = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_PKG, "libgpufs.so")
+
+COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", "writeback", "rpc",
+            "rpc_open", "rpc_read", "rpc_write", "bytes_h2d", "bytes_d2h", "open_fast", "reopen_valid",
+            "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
+            "ring_wait"]
+HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
+                 "errors", "merges"]
+
+O_RDONLY = 0
+O_GWRONCE = 1
+F_LOCKED_TRAVERSAL = 1
+F_NO_DMA_COMPLETION = 2
+DAEMON_SPAWN = 0
+DAEMON_RUN = 1
+
+
+class GfsError(OSError):
+    pass
+
+
+class gfs_config(ctypes.Structure):
+    _fields_ = [("device", ctypes.c_int), ("cache_bytes", ctypes.c_uint64), ("page_size", ctypes.c_uint32),
+                ("ring_slots", ctypes.c_uint32), ("daemon_threads", ctypes.c_uint32),
+                ("max_files", ctypes.c_uint32), ("max_nodes", ctypes.c_uint32), ("max_batch", ctypes.c_uint32),
+                ("flags", ctypes.c_uint32), ("pad", ctypes.c_uint32), ("timeout_ms", ctypes.c_uint64),
+                ("frame_pool", ctypes.c_void_p)]
+
+
+_lib = None
+
+
+def lib():
+    """Load libgpufs.so (built in-tree by build.py / __graft_entry__.build())."""
+    global _lib
+    if _lib is None:
+        if not os.path.exists(LIB_PATH):
+            raise ImportError(f"{LIB_PATH} is missing: run `python -m paper_conf_asplos_silbersteinfkw13_b200.build`"
+                              " (there is no CPU fallback)")
+        L = ctypes.CDLL(LIB_PATH)
+        P, I, U32, U64 = ctypes.c_void_p, ctypes.c_int, ctypes.c_uint32, ctypes.c_uint64
+        CS = ctypes.c_char_p
+        sig = {
+            "gfs_config_default": ([ctypes.POINTER(gfs_config)], I),
+            "gfs_init": ([ctypes.POINTER(gfs_config), ctypes.POINTER(P)], I),
+            "gfs_daemon": ([P, I], I),
+            "gfs_daemon_stop": ([P], I),
+            "gfs_shutdown": ([P], I),
+            "gfs_device_ctx": ([P], P),
+            "gfs_stats": ([P, P, I, I], I),
+            "gfs_host_stats": ([P, P, I], I),
+            "gfs_info": ([P, P, I], I),
+            "gfs_run_gread": ([P, P, CS, I, U32, P, P, P, P, P, U32, U32, U32], I),
+            "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
+            "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
+            "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32], I),
+            "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
+        }
+        for name, (args, res) in sig.items():
+            fn = getattr(L, name)
+            fn.argtypes = args
+            fn.restype = res
+        _lib = L
+    return _lib
+
+
+def _ck(r: int, what: str) -> int:
+    if r < 0:
+        raise GfsError(-r, f"{what}: {os.strerror(-r)}")
+    return r
+
+
+def _b(path) -> bytes:
+    return os.fsencode(path)
+
+
+# ------------------------------------------------------------------ host API
+def gfs_config_default(**kw) -> gfs_config:
+    c = gfs_config()
+    _ck(lib().gfs_config_default(ctypes.byref(c)), "gfs_config_default")
+    for k, v in kw.items():
+        setattr(c, k, v)
+    return c
+
+
+def gfs_init(cfg: gfs_config) -> int:
+    h = ctypes.c_void_p()
+    _ck(lib().gfs_init(ctypes.byref(cfg), ctypes.byref(h)), "gfs_init")
+    return h.value
+
+
+def gfs_daemon(h: int, mode: int = DAEMON_SPAWN) -> int:
+    return _ck(lib().gfs_daemon(h, mode), "gfs_daemon")
+
+
+def gfs_daemon_stop(h: int) -> int:
+    return _ck(lib().gfs_daemon_stop(h), "gfs_daemon_stop")
+
+
+def gfs_shutdown(h: int) -> int:
+    return _ck(lib().gfs_shutdown(h), "gfs_shutdown")
+
+
+def gfs_device_ctx(h: int) -> int:
+    return lib().gfs_device_ctx(h)
+
+
+def gfs_stats(h: int, reset: bool = False) -> dict:
+    a = (ctypes.c_uint64 * len(COUNTERS))()
+    _ck(lib().gfs_stats(h, a, len(COUNTERS), 1 if reset else 0), "gfs_stats")
+    return dict(zip(COUNTERS, (int(x) for x in a)))
+
+
+def gfs_host_stats(h: int) -> dict:
+    a = (ctypes.c_uint64 * len(HOST_COUNTERS))()
+    _ck(lib().gfs_host_stats(h, a, len(HOST_COUNTERS)), "gfs_host_stats")
+    return dict(zip(HOST_COUNTERS, (int(x) for x in a)))
+
+
+def gfs_info(h: int) -> dict:
+    a = (ctypes.c_uint64 * 7)()
+    _ck(lib().gfs_info(h, a, 7), "gfs_info")
+    return dict(zip(["page_size", "nframes", "max_files", "max_nodes", "ring_slots", "daemon_threads",
+                     "stream_write_value64"], (int(x) for x in a)))
+
+
+# ------------------------------------------------------------------ launchers
+def gfs_run_gread(h, stream, path, mode, ncalls, d_off, d_len, d_dstoff, d_dst, d_ret, grid, block, smem=0):
+    return _ck(lib().gfs_run_gread(h, stream, _b(path), mode, ncalls, d_off, d_len, d_dstoff, d_dst, d_ret,
+                                   grid, block, smem), "gfs_run_gread")
+
+
+def gfs_run_seqread(h, stream, path, file_off, total, chunk, use_mmap, d_scratch, d_sum, d_err, grid, block):
+    return _ck(lib().gfs_run_seqread(h, stream, _b(path), file_off, total, chunk, use_mmap, d_scratch, d_sum,
+                                     d_err, grid, block), "gfs_run_seqread")
+
+
+def gfs_run_randread(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):
+    return _ck(lib().gfs_run_randread(h, stream, _b(path) if path else None, raw, d_raw, chunk, calls_per_block,
+                                      d_off, d_sum, d_err, grid, block), "gfs_run_randread")
+
+
+def gfs_run_gwrite(h, stream, path, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid, block):
+    return _ck(lib().gfs_run_gwrite(h, stream, _b(path), ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid,
+                                    block), "gfs_run_gwrite")
+
+
+def gfs_run_fileop(h, stream, path, flags, op, arg, d_ret):
+    return _ck(lib().gfs_run_fileop(h, stream, _b(path), flags, op, arg, d_ret), "gfs_run_fileop")
+
+
+from . import build  # noqa: E402,F401
+from .api import GpuFS  # noqa: E402  (torch-facing convenience wrapper)

@@ -1,0 +1,179 @@
+"""Torch-facing convenience wrapper over the C ABI (marshalling only).
+
+torch supplies device memory and the CUDA stream; every operation is one
+launcher of libgpufs.so. Methods synchronise the stream before returning
+results unless ``sync=False``.
+"""
+from __future__ import annotations
+
+import numpy as np
+
+from . import (DAEMON_SPAWN, gfs_config_default, gfs_daemon, gfs_daemon_stop, gfs_host_stats, gfs_info,
+               gfs_init, gfs_run_fileop, gfs_run_gread, gfs_run_gwrite, gfs_run_randread, gfs_run_seqread,
+               gfs_shutdown, gfs_stats, gfs_device_ctx)
+
+
+def _torch():
+    import torch
+    if not torch.cuda.is_available():
+        raise RuntimeError("GpuFS needs a CUDA device (there is no CPU fallback)")
+    return torch
+
+
+class GpuFS:
+    """One GPU buffer cache + its host daemon (gfs_init + gfs_daemon)."""
+
+    def __init__(self, cache_bytes=1 << 30, page_size=64 << 10, device=0, daemon_threads=8, ring_slots=4096,
+                 max_files=4096, max_nodes=0, max_batch=32, flags=0, timeout_ms=60000):
+        torch = _torch()
+        torch.cuda.set_device(device)
+        self.device = device
+        self.page_size = page_size
+        cfg = gfs_config_default(device=device, cache_bytes=cache_bytes, page_size=page_size,
+                                 daemon_threads=daemon_threads, ring_slots=ring_slots, max_files=max_files,
+                                 max_nodes=max_nodes, max_batch=max_batch, flags=flags, timeout_ms=timeout_ms)
+        self.h = gfs_init(cfg)
+        gfs_daemon(self.h, DAEMON_SPAWN)
+
+    # lifecycle --------------------------------------------------------------
+    def close(self):
+        if getattr(self, "h", None):
+            _torch().cuda.synchronize(self.device)
+            gfs_shutdown(self.h)
+            self.h = None
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.close()
+
+    def stop_daemon(self):
+        gfs_daemon_stop(self.h)
+
+    def start_daemon(self):
+        gfs_daemon(self.h, DAEMON_SPAWN)
+
+    def stats(self, reset=False) -> dict:
+        return gfs_stats(self.h, reset)
+
+    def host_stats(self) -> dict:
+        return gfs_host_stats(self.h)
+
+    def info(self) -> dict:
+        return gfs_info(self.h)
+
+    @property
+    def ctx(self) -> int:
+        return gfs_device_ctx(self.h)
+
+    # helpers ----------------------------------------------------------------
+    def _stream(self, stream=None):
+        torch = _torch()
+        s = stream if stream is not None else torch.cuda.current_stream(self.device)
+        return s, s.cuda_stream
+
+    def _dev(self, a, dtype=None):
+        torch = _torch()
+        return torch.as_tensor(np.ascontiguousarray(a), device=f"cuda:{self.device}", dtype=dtype)
+
+    # gread / gmmap parity harness -------------------------------------------
+    def gread_calls(self, path, offs, lens, mode=0, grid=None, block=256, smem=0, stream=None):
+        """Issue gread (mode 0), gmmap (1) or gread-to-shared (2) calls; returns (ret, dst, dstoff)."""
+        torch = _torch()
+        offs = np.asarray(offs, dtype=np.uint64)
+        lens = np.asarray(lens, dtype=np.uint64)
+        n = len(offs)
+        dstoff = np.concatenate([[0], np.cumsum(lens)[:-1]]).astype(np.uint64) if n else np.zeros(0, np.uint64)
+        total = int(lens.sum()) if n else 0
+        d_off = self._dev(offs.view(np.int64))
+        d_len = self._dev(lens.view(np.int64))
+        d_dstoff = self._dev(dstoff.view(np.int64))
+        d_dst = torch.zeros(max(total, 1), dtype=torch.uint8, device=f"cuda:{self.device}")
+        d_ret = torch.full((max(n, 1),), -999, dtype=torch.int64, device=f"cuda:{self.device}")
+        s, sp = self._stream(stream)
+        grid = grid or max(1, min(n, 296))
+        if mode == 2 and smem == 0:
+            smem = int(lens.max()) if n else 16
+            smem = (smem + 15) // 16 * 16
+        gfs_run_gread(self.h, sp, path, mode, n, d_off.data_ptr(), d_len.data_ptr(), d_dstoff.data_ptr(),
+                      d_dst.data_ptr(), d_ret.data_ptr(), grid, block, smem)
+        s.synchronize()
+        return d_ret[:n].cpu().numpy(), d_dst.cpu().numpy(), dstoff
+
+    # sequential sweep (C2 / K1) ---------------------------------------------
+    def seqread(self, path, total, chunk, file_off=0, use_mmap=False, grid=296, block=256, stream=None,
+                sync=True, scratch=None, out=None):
+        torch = _torch()
+        dev = f"cuda:{self.device}"
+        if scratch is None:
+            scratch = torch.empty(max(1, grid * chunk if not use_mmap else 1), dtype=torch.uint8, device=dev)
+        if out is None:
+            out = torch.zeros(2, dtype=torch.int64, device=dev)  # [sum, err]
+        s, sp = self._stream(stream)
+        gfs_run_seqread(self.h, sp, path, file_off, total, chunk, 1 if use_mmap else 0, scratch.data_ptr(),
+                        out.data_ptr(), out.data_ptr() + 8, grid, block)
+        if not sync:
+            return out
+        s.synchronize()
+        v = out.cpu().numpy()
+        return int(v[0].astype(np.uint64)), int(v[1])
+
+    # cache-hit reads into shared memory (K4) ---------------------------------
+    def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None):
+        torch = _torch()
+        dev = f"cuda:{self.device}"
+        offs = np.asarray(offs, dtype=np.uint64)
+        assert len(offs) % grid == 0
+        calls = len(offs) // grid
+        d_off = offs if isinstance(offs, torch.Tensor) else self._dev(offs.view(np.int64))
+        if out is None:
+            out = torch.zeros(2, dtype=torch.int64, device=dev)
+        s, sp = self._stream(stream)
+        gfs_run_randread(self.h, sp, path, 1 if raw is not None else 0,
+                         raw.data_ptr() if raw is not None else None, chunk, calls, d_off.data_ptr(),
+                         out.data_ptr(), out.data_ptr() + 8, grid, block)
+        if not sync:
+            return out
+        s.synchronize()
+        v = out.cpu().numpy()
+        return int(v[0].astype(np.uint64)), int(v[1])
+
+    # gwrite -----------------------------------------------------------------
+    def gwrite_calls(self, path, offs, lens, data: bytes, srcoff=None, grid=None, block=256, stream=None):
+        torch = _torch()
+        offs = np.asarray(offs, dtype=np.uint64)
+        lens = np.asarray(lens, dtype=np.uint64)
+        n = len(offs)
+        if srcoff is None:
+            srcoff = np.concatenate([[0], np.cumsum(lens)[:-1]]).astype(np.uint64) if n else np.zeros(0, np.uint64)
+        src = np.frombuffer(bytes(data), dtype=np.uint8) if len(data) else np.zeros(1, np.uint8)
+        d_src = self._dev(src)
+        d_off = self._dev(offs.view(np.int64))
+        d_len = self._dev(lens.view(np.int64))
+        d_srcoff = self._dev(np.asarray(srcoff, np.uint64).view(np.int64))
+        d_ret = torch.full((max(n, 1),), -999, dtype=torch.int64, device=f"cuda:{self.device}")
+        s, sp = self._stream(stream)
+        gfs_run_gwrite(self.h, sp, path, n, d_off.data_ptr(), d_len.data_ptr(), d_srcoff.data_ptr(),
+                       d_src.data_ptr(), d_ret.data_ptr(), grid or max(1, min(n, 296)), block)
+        s.synchronize()
+        return d_ret[:n].cpu().numpy()
+
+    def fileop(self, path, op, flags=0, arg=0, stream=None) -> int:
+        """op: 'fsync' | 'ftruncate' | 'fstat' | 'openclose'."""
+        torch = _torch()
+        code = {"fsync": 0, "ftruncate": 1, "fstat": 2, "openclose": 3}[op]
+        d_ret = torch.full((1,), -999, dtype=torch.int64, device=f"cuda:{self.device}")
+        s, sp = self._stream(stream)
+        gfs_run_fileop(self.h, sp, path, flags, code, arg, d_ret.data_ptr())
+        s.synchronize()
+        return int(d_ret.item())
+
+    def gfsync(self, path):
+        return self.fileop(path, "fsync", flags=1)
+
+    def gftruncate(self, path, size):
+        return self.fileop(path, "ftruncate", flags=1, arg=size)
+
+    def gfstat(self, path, flags=0):
+        return self.fileop(path, "fstat", flags=flags)

@@ -1,0 +1,661 @@
+// gfs_host.cpp — host runtime of libgpufs.so: gfs_init / gfs_daemon / stats.
+//
+// The host side of GPUfs ("a user-level thread in the host
+// application, giving it access to the application's CUDA context") and of the
+// GPU-as-client RPC (§4.3). B200 redesign:
+//   * the request queue is a ring of 64-byte slots in pinned, mapped host
+//     memory, one queue per GPU owned by that GPU; a slot is
+//     published by the GPU with st.release.sys on its seq word;
+//   * W worker threads (not the paper's single event thread) each
+//     claim the next ticket, spin on its slot, pread into a pinned staging
+//     buffer (double-buffered per worker) and cudaMemcpyAsync it into the
+//     cache frame on the worker's own non-blocking stream;
+//   * completion is stream-ordered after the DMA: cuStreamWriteValue64 of
+//     ((ticket+1) << 32 | result) into a completion word in HBM, which the
+//     waiting GPU thread polls locally (no PCIe reads on the GPU side);
+//   * dirty ranges come back by D2H + pwrite; a partially written range is
+//     merged with the host copy by "diff against zeros";
+//   * close-to-open consistency uses a shared-memory version table keyed by
+//     (st_dev, st_ino), bumped on every write-back (stand-in for WRAPFS,
+//     P:L760-772); OPEN replies carry it so re-opens can validate.
+#include <atomic>
+#include <cerrno>
+#include <chrono>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <fcntl.h>
+#include <mutex>
+#include <sched.h>
+#include <string>
+#include <sys/mman.h>
+#include <sys/stat.h>
+#include <thread>
+#include <unistd.h>
+#include <vector>
+
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include "gpufs.h"
+
+#define GFS_API extern "C" __attribute__((visibility("default")))
+
+// Launchers live in gfs_kernels.cu; they need these.
+extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s);
+
+namespace {
+
+typedef CUresult (*PFN_writeValue64)(CUstream, CUdeviceptr, cuuint64_t, unsigned int);
+typedef CUresult (*PFN_devAttr)(int*, CUdevice_attribute, CUdevice);
+
+inline void cpu_relax() {
+#if defined(__x86_64__)
+  __builtin_ia32_pause();
+#endif
+}
+
+int64_t pread_full(int fd, uint8_t* buf, uint64_t len, uint64_t off) {
+  uint64_t done = 0;
+  while (done < len) {
+    ssize_t r = pread(fd, buf + done, len - done, (off_t)(off + done));
+    if (r < 0) {
+      if (errno == EINTR) continue;
+      return -errno;
+    }
+    if (r == 0) break;
+    done += (uint64_t)r;
+  }
+  return (int64_t)done;
+}
+
+int64_t pwrite_full(int fd, const uint8_t* buf, uint64_t len, uint64_t off) {
+  uint64_t done = 0;
+  while (done < len) {
+    ssize_t r = pwrite(fd, buf + done, len - done, (off_t)(off + done));
+    if (r < 0) {
+      if (errno == EINTR) continue;
+      return -errno;
+    }
+    done += (uint64_t)r;
+  }
+  return (int64_t)done;
+}
+
+// ---------------------------------------------------------------- version table
+// Shared by every process on the host (one per GPU): open addressing over
+// 64-bit keys mixed from (st_dev, st_ino); version bumped per write-back.
+struct VEntry {
+  uint64_t key;
+  uint64_t version;
+};
+constexpr uint64_t kVEntries = 1u << 16;
+
+struct VersionTable {
+  VEntry* e = nullptr;
+  bool open() {
+    const char* name = getenv("GFS_VERSION_TABLE");
+    std::string path = name && *name ? name : "/dev/shm/gfs_version_table_v1";
+    int fd = ::open(path.c_str(), O_RDWR | O_CREAT, 0666);
+    if (fd < 0) return false;
+    const size_t bytes = kVEntries * sizeof(VEntry);
+    struct stat st;
+    if (fstat(fd, &st) != 0) { ::close(fd); return false; }
+    if ((size_t)st.st_size < bytes && ftruncate(fd, (off_t)bytes) != 0) { ::close(fd); return false; }
+    void* p = mmap(nullptr, bytes, PROT_READ | PROT_WRITE, MAP_SHARED, fd, 0);
+    ::close(fd);
+    if (p == MAP_FAILED) return false;
+    e = (VEntry*)p;
+    return true;
+  }
+  void close() {
+    if (e) munmap(e, kVEntries * sizeof(VEntry));
+    e = nullptr;
+  }
+  static uint64_t mix(uint64_t dev, uint64_t ino) {
+    uint64_t z = dev * 0x9E3779B97F4A7C15ull ^ (ino + 0x632BE59BD9B4E019ull);
+    z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+    z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+    z ^= z >> 31;
+    return z | 1;
+  }
+  VEntry* find(uint64_t dev, uint64_t ino, bool create) {
+    if (!e) return nullptr;
+    const uint64_t k = mix(dev, ino);
+    for (uint64_t i = 0; i < kVEntries; ++i) {
+      VEntry* x = e + ((k + i) & (kVEntries - 1));
+      uint64_t cur = __atomic_load_n(&x->key, __ATOMIC_ACQUIRE);
+      if (cur == k) return x;
+      if (cur == 0) {
+        if (!create) return nullptr;
+        uint64_t zero = 0;
+        if (__atomic_compare_exchange_n(&x->key, &zero, k, false, __ATOMIC_ACQ_REL, __ATOMIC_ACQUIRE)) return x;
+        if (zero == k) return x;
+      }
+    }
+    return nullptr;
+  }
+  uint64_t get(uint64_t dev, uint64_t ino) {
+    VEntry* x = find(dev, ino, false);
+    return x ? __atomic_load_n(&x->version, __ATOMIC_ACQUIRE) : 0;
+  }
+  void bump(uint64_t dev, uint64_t ino) {
+    VEntry* x = find(dev, ino, true);
+    if (x) __atomic_fetch_add(&x->version, 1, __ATOMIC_ACQ_REL);
+  }
+};
+
+enum {
+  HS_RPC = 0, HS_READ, HS_WRITE, HS_OPEN, HS_CLOSE, HS_TRUNC, HS_BYTES_H2D, HS_BYTES_D2H, HS_PREAD_NS,
+  HS_ERRORS, HS_MERGES, HS_N
+};
+
+}  // namespace
+
+struct HostFile {
+  int fd = -1;
+  uint32_t mode = 0;
+  uint64_t dev = 0, ino = 0;
+};
+
+struct gfs_handle;
+
+struct Worker {
+  std::thread th;
+  cudaStream_t stream = nullptr;
+  uint8_t* staging[2] = {nullptr, nullptr};
+  cudaEvent_t ev[2] = {nullptr, nullptr};
+  bool pending[2] = {false, false};
+  int cur = 0;
+  std::vector<uint8_t> merge;
+};
+
+struct gfs_handle {
+  gfs_config cfg{};
+  gfs_ctx h{};         // host copy holding device pointers
+  gfs_ctx* d = nullptr;  // device copy
+  bool own_pool = false;
+  cudaStream_t priv = nullptr;
+  gfs_rpc_req* ring_h = nullptr;
+  gfs_rpc_resp* resp_h = nullptr;
+  char* paths_h = nullptr;
+  uint64_t* cplsrc_h = nullptr;
+  std::vector<Worker> workers;
+  std::atomic<uint64_t> next_ticket{0};
+  std::atomic<bool> running{false};
+  std::thread runner_dummy;
+  std::mutex fd_mu;
+  std::vector<HostFile> files;
+  std::vector<uint32_t> free_hfids;
+  PFN_writeValue64 wv64 = nullptr;
+  VersionTable vt;
+  std::atomic<uint64_t> hs[HS_N];
+  uint64_t staging_bytes = 0;
+};
+
+namespace {
+
+int cuda_err(cudaError_t e) {
+  if (e == cudaSuccess) return 0;
+  if (e == cudaErrorMemoryAllocation) return -ENOMEM;
+  return -EIO;
+}
+
+#define CK(x)                         \
+  do {                                \
+    cudaError_t _e = (x);             \
+    if (_e != cudaSuccess) {          \
+      fprintf(stderr, "gpufs: %s failed: %s\n", #x, cudaGetErrorString(_e)); \
+      rc = cuda_err(_e);              \
+      goto fail;                      \
+    }                                 \
+  } while (0)
+
+uint32_t alloc_hfid(gfs_handle* h, const HostFile& f) {
+  std::lock_guard<std::mutex> g(h->fd_mu);
+  if (!h->free_hfids.empty()) {
+    uint32_t id = h->free_hfids.back();
+    h->free_hfids.pop_back();
+    h->files[id] = f;
+    return id;
+  }
+  h->files.push_back(f);
+  return (uint32_t)(h->files.size() - 1);
+}
+
+HostFile get_hfid(gfs_handle* h, uint32_t id) {
+  std::lock_guard<std::mutex> g(h->fd_mu);
+  if (id >= h->files.size()) return HostFile();
+  return h->files[id];
+}
+
+void free_hfid(gfs_handle* h, uint32_t id) {
+  std::lock_guard<std::mutex> g(h->fd_mu);
+  if (id >= h->files.size() || h->files[id].fd < 0) return;
+  ::close(h->files[id].fd);
+  h->files[id] = HostFile();
+  h->free_hfids.push_back(id);
+}
+
+void complete(gfs_handle* h, Worker& w, uint32_t slot, uint64_t ticket, int32_t result) {
+  const uint64_t v = ((ticket + 1) << 32) | (uint32_t)result;
+  CUdeviceptr addr = (CUdeviceptr)(h->h.cpl + slot);
+  if (h->wv64) {
+    CUresult r = h->wv64((CUstream)w.stream, addr, v, 0);
+    if (r == CUDA_SUCCESS) return;
+  }
+  // Fallback: an 8-byte H2D copy from a per-slot pinned source, ordered after the DMA.
+  h->cplsrc_h[slot] = v;
+  cudaMemcpyAsync((void*)addr, &h->cplsrc_h[slot], 8, cudaMemcpyHostToDevice, w.stream);
+}
+
+uint8_t* staging_acquire(Worker& w) {
+  const int b = w.cur;
+  if (w.pending[b]) {
+    cudaEventSynchronize(w.ev[b]);
+    w.pending[b] = false;
+  }
+  return w.staging[b];
+}
+void staging_issued(Worker& w) {
+  cudaEventRecord(w.ev[w.cur], w.stream);
+  w.pending[w.cur] = true;
+  w.cur ^= 1;
+}
+
+int32_t do_open(gfs_handle* h, uint32_t slot, const gfs_rpc_req& q) {
+  gfs_rpc_resp* rs = h->resp_h + slot;
+  std::string path(h->paths_h + (size_t)slot * GFS_MAX_PATH, q.path_len < GFS_MAX_PATH ? q.path_len : 0);
+  const bool gw = (q.flags & GFS_O_GWRONCE) != 0;
+  int fd = ::open(path.c_str(), gw ? (O_RDWR | O_CREAT) : O_RDONLY, 0644);
+  if (fd < 0) {
+    rs->status = -errno;
+    return rs->status;
+  }
+  struct stat st;
+  if (fstat(fd, &st) != 0) {
+    rs->status = -errno;
+    ::close(fd);
+    return rs->status;
+  }
+  uint32_t hfid;
+  bool reused = false;
+  if (q.arg) {  // re-open of a cached file: keep its host fd if it is the same file
+    const uint32_t old = (uint32_t)(q.arg - 1);
+    HostFile of = get_hfid(h, old);
+    if (of.fd >= 0 && of.dev == (uint64_t)st.st_dev && of.ino == (uint64_t)st.st_ino &&
+        (of.mode & GFS_O_GWRONCE) >= (q.flags & GFS_O_GWRONCE)) {
+      ::close(fd);
+      hfid = old;
+      reused = true;
+    } else {
+      free_hfid(h, old);
+    }
+  }
+  if (!reused) {
+    HostFile f;
+    f.fd = fd;
+    f.mode = q.flags;
+    f.dev = st.st_dev;
+    f.ino = st.st_ino;
+    hfid = alloc_hfid(h, f);
+  }
+  rs->size = (int64_t)st.st_size;
+  rs->version = h->vt.get(st.st_dev, st.st_ino);
+  rs->ino = st.st_ino;
+  rs->dev = st.st_dev;
+  rs->mtime_ns = (int64_t)st.st_mtim.tv_sec * 1000000000ll + st.st_mtim.tv_nsec;
+  rs->hfid = hfid;
+  rs->status = 0;
+  h->hs[HS_OPEN]++;
+  return 0;
+}
+
+int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
+  HostFile f = get_hfid(h, q.hfid);
+  if (f.fd < 0) return -EBADF;
+  if (q.len > h->staging_bytes) return -EINVAL;
+  uint8_t* buf = staging_acquire(w);
+  auto t0 = std::chrono::steady_clock::now();
+  int64_t n = pread_full(f.fd, buf, q.len, q.file_off);
+  h->hs[HS_PREAD_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
+                            std::chrono::steady_clock::now() - t0).count();
+  if (n < 0) return (int32_t)n;
+  if ((uint64_t)n < q.len) memset(buf + n, 0, q.len - (size_t)n);  // host file shrank: zeros (R4)
+  if (q.len) {
+    cudaError_t e = cudaMemcpyAsync((void*)q.dev_ptr, buf, q.len, cudaMemcpyHostToDevice, w.stream);
+    if (e != cudaSuccess) return -EIO;
+    staging_issued(w);
+  }
+  h->hs[HS_READ]++;
+  h->hs[HS_BYTES_H2D] += q.len;
+  return (int32_t)q.len;
+}
+
+int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
+  HostFile f = get_hfid(h, q.hfid);
+  if (f.fd < 0) return -EBADF;
+  if (!(f.mode & GFS_O_GWRONCE)) return -EBADF;  // read-only files are never written back
+  if (q.len > h->staging_bytes) return -EINVAL;
+  uint8_t* buf = staging_acquire(w);
+  if (q.len) {
+    if (cudaMemcpyAsync(buf, (const void*)q.dev_ptr, q.len, cudaMemcpyDeviceToHost, w.stream) != cudaSuccess)
+      return -EIO;
+    if (cudaStreamSynchronize(w.stream) != cudaSuccess) return -EIO;
+  }
+  if (!(q.flags & GFS_WF_FULL)) {
+    // Not every byte of the range was written: diff against zeros.
+    w.merge.assign(q.len, 0);
+    int64_t r = pread_full(f.fd, w.merge.data(), q.len, q.file_off);
+    if (r < 0) return (int32_t)r;
+    for (uint32_t i = 0; i < q.len; ++i)
+      if (buf[i] == 0) buf[i] = w.merge[i];
+    h->hs[HS_MERGES]++;
+  }
+  int64_t r = pwrite_full(f.fd, buf, q.len, q.file_off);
+  if (r < 0) return (int32_t)r;
+  h->vt.bump(f.dev, f.ino);
+  h->hs[HS_WRITE]++;
+  h->hs[HS_BYTES_D2H] += q.len;
+  return (int32_t)q.len;
+}
+
+void worker_loop(gfs_handle* h, int wi) {
+  cudaSetDevice(h->cfg.device);
+  Worker& w = h->workers[wi];
+  const uint32_t R = h->h.ring_slots;
+  while (h->running.load(std::memory_order_acquire)) {
+    const uint64_t t = h->next_ticket.fetch_add(1);
+    const uint32_t slot = (uint32_t)(t % R);
+    volatile gfs_rpc_req* vq = h->ring_h + slot;
+    uint64_t spins = 0;
+    bool stop = false;
+    while (__atomic_load_n((const uint64_t*)&vq->seq, __ATOMIC_ACQUIRE) != t + 1) {
+      if (!h->running.load(std::memory_order_relaxed)) {
+        stop = true;
+        break;
+      }
+      ++spins;
+      if (spins < 4096) {
+        cpu_relax();
+      } else if (spins < 65536) {
+        sched_yield();
+      } else {
+        usleep(50);
+      }
+    }
+    if (stop) break;
+    gfs_rpc_req q;
+    q.op = vq->op;
+    q.hfid = vq->hfid;
+    q.file_off = vq->file_off;
+    q.dev_ptr = vq->dev_ptr;
+    q.len = vq->len;
+    q.flags = vq->flags;
+    q.arg = vq->arg;
+    q.path_len = vq->path_len;
+    int32_t res;
+    switch (q.op) {
+      case GFS_OP_READ: res = do_read(h, w, q); break;
+      case GFS_OP_WRITE: res = do_write(h, w, q); break;
+      case GFS_OP_OPEN: res = do_open(h, slot, q); break;
+      case GFS_OP_CLOSE:
+        free_hfid(h, q.hfid);
+        h->hs[HS_CLOSE]++;
+        res = 0;
+        break;
+      case GFS_OP_TRUNC: {
+        HostFile f = get_hfid(h, q.hfid);
+        res = f.fd < 0 ? -EBADF : (ftruncate(f.fd, (off_t)q.arg) == 0 ? 0 : -errno);
+        if (res == 0) h->vt.bump(f.dev, f.ino);
+        h->hs[HS_TRUNC]++;
+        break;
+      }
+      case GFS_OP_NOP: res = 0; break;
+      default: res = -ENOSYS;
+    }
+    if (res < 0) h->hs[HS_ERRORS]++;
+    h->hs[HS_RPC]++;
+    complete(h, w, slot, t, res);
+  }
+  cudaStreamSynchronize(w.stream);
+}
+
+void free_all(gfs_handle* h) {
+  auto F = [](void* p) {
+    if (p) cudaFree(p);
+  };
+  if (h->own_pool) F(h->h.pool);
+  F(h->h.f_state); F(h->h.f_tag); F(h->h.f_file); F(h->h.f_valid); F(h->h.f_lo); F(h->h.f_hi);
+  F(h->h.f_written); F(h->h.f_stamp); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
+  F(h->h.node_free); F(h->h.node_free_top); F(h->h.node_lock); F(h->h.files); F(h->h.paths); F(h->h.uid_next);
+  F(h->h.cpl); F(h->h.ack); F(h->h.ring_tail); F(h->h.ctr); F(h->d);
+  if (h->ring_h) cudaFreeHost(h->ring_h);
+  if (h->resp_h) cudaFreeHost(h->resp_h);
+  if (h->paths_h) cudaFreeHost(h->paths_h);
+  if (h->cplsrc_h) cudaFreeHost(h->cplsrc_h);
+  for (auto& w : h->workers) {
+    for (int b = 0; b < 2; ++b) {
+      if (w.staging[b]) cudaFreeHost(w.staging[b]);
+      if (w.ev[b]) cudaEventDestroy(w.ev[b]);
+    }
+    if (w.stream) cudaStreamDestroy(w.stream);
+  }
+  if (h->priv) cudaStreamDestroy(h->priv);
+  for (auto& f : h->files)
+    if (f.fd >= 0) ::close(f.fd);
+  h->vt.close();
+}
+
+bool pow2(uint64_t x) { return x && !(x & (x - 1)); }
+
+}  // namespace
+
+GFS_API int gfs_config_default(gfs_config* c) {
+  if (!c) return -EINVAL;
+  memset(c, 0, sizeof(*c));
+  c->device = 0;
+  c->cache_bytes = 1ull << 30;
+  c->page_size = 64u << 10;
+  c->ring_slots = 4096;
+  c->daemon_threads = 8;
+  c->max_files = 4096;
+  c->max_nodes = 0;
+  c->max_batch = GFS_MAX_BATCH;
+  c->flags = 0;
+  c->timeout_ms = 60000;
+  return 0;
+}
+
+GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
+  if (!cfg || !out) return -EINVAL;
+  if (!pow2(cfg->page_size) || cfg->page_size < 4096 || cfg->page_size > (16u << 20)) return -EINVAL;
+  if (!pow2(cfg->ring_slots) || !pow2(cfg->max_files)) return -EINVAL;
+  if (cfg->daemon_threads == 0 || cfg->daemon_threads > 256) return -EINVAL;
+  const uint64_t nframes = cfg->cache_bytes / cfg->page_size;
+  if (nframes == 0 || nframes >= (1ull << 31)) return -EINVAL;
+  int ndev = 0;
+  if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev == 0) return -ENODEV;
+  if (cfg->device < 0 || cfg->device >= ndev) return -ENODEV;
+
+  gfs_handle* h = new gfs_handle();
+  for (auto& x : h->hs) x = 0;
+  h->cfg = *cfg;
+  int rc = 0;
+  gfs_ctx& c = h->h;
+  const uint32_t R = cfg->ring_slots;
+  const uint32_t MF = cfg->max_files;
+  uint32_t max_nodes = cfg->max_nodes ? cfg->max_nodes : (MF * 2u + 65536u);
+  size_t ctr_bytes = (size_t)GFS_C_NCOUNTERS * GFS_CTR_SHARDS * sizeof(unsigned long long);
+
+  CK(cudaSetDevice(cfg->device));
+  CK(cudaFree(0));
+  CK(cudaStreamCreateWithFlags(&h->priv, cudaStreamNonBlocking));
+  c.page_size = cfg->page_size;
+  c.page_shift = (uint32_t)__builtin_ctz(cfg->page_size);
+  c.nframes = (uint32_t)nframes;
+  if (cfg->frame_pool) {
+    c.pool = (uint8_t*)cfg->frame_pool;
+  } else {
+    CK(cudaMalloc((void**)&c.pool, nframes * cfg->page_size));
+    h->own_pool = true;
+  }
+  CK(cudaMalloc((void**)&c.f_state, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_tag, nframes * 8));
+  CK(cudaMalloc((void**)&c.f_file, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_valid, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_lo, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_hi, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_written, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_stamp, nframes * 4));
+  CK(cudaMalloc((void**)&c.fresh_next, 4));
+  CK(cudaMalloc((void**)&c.hand, 4));
+  c.max_nodes = max_nodes;
+  CK(cudaMalloc((void**)&c.nodes, (size_t)max_nodes * GFS_FANOUT * 4));
+  CK(cudaMalloc((void**)&c.node_next, 4));
+  CK(cudaMalloc((void**)&c.node_free, (size_t)max_nodes * 4));
+  CK(cudaMalloc((void**)&c.node_free_top, 4));
+  CK(cudaMalloc((void**)&c.node_lock, 4));
+  c.max_files = MF;
+  CK(cudaMalloc((void**)&c.files, (size_t)MF * sizeof(gfs_file)));
+  CK(cudaMalloc((void**)&c.paths, (size_t)MF * GFS_MAX_PATH));
+  CK(cudaMalloc((void**)&c.uid_next, 4));
+  c.ring_slots = R;
+  CK(cudaHostAlloc((void**)&h->ring_h, (size_t)R * sizeof(gfs_rpc_req), cudaHostAllocMapped | cudaHostAllocPortable));
+  CK(cudaHostAlloc((void**)&h->resp_h, (size_t)R * sizeof(gfs_rpc_resp), cudaHostAllocMapped | cudaHostAllocPortable));
+  CK(cudaHostAlloc((void**)&h->paths_h, (size_t)R * GFS_MAX_PATH, cudaHostAllocMapped | cudaHostAllocPortable));
+  CK(cudaHostAlloc((void**)&h->cplsrc_h, (size_t)R * 8, cudaHostAllocPortable));
+  memset(h->ring_h, 0, (size_t)R * sizeof(gfs_rpc_req));
+  memset(h->resp_h, 0, (size_t)R * sizeof(gfs_rpc_resp));
+  CK(cudaHostGetDevicePointer((void**)&c.ring, h->ring_h, 0));
+  CK(cudaHostGetDevicePointer((void**)&c.resp, h->resp_h, 0));
+  CK(cudaHostGetDevicePointer((void**)&c.ring_paths, h->paths_h, 0));
+  CK(cudaMalloc((void**)&c.cpl, (size_t)R * 8));
+  CK(cudaMalloc((void**)&c.ack, (size_t)R * 8));
+  CK(cudaMalloc((void**)&c.ring_tail, 8));
+  CK(cudaMalloc((void**)&c.ctr, ctr_bytes));
+  c.flags = cfg->flags;
+  c.max_batch = cfg->max_batch >= 1 && cfg->max_batch <= GFS_MAX_BATCH ? cfg->max_batch : GFS_MAX_BATCH;
+  c.timeout_ns = cfg->timeout_ms * 1000000ull;
+  CK(cudaMemsetAsync(c.nodes, 0, (size_t)max_nodes * GFS_FANOUT * 4, h->priv));
+  CK(cudaMemsetAsync(c.files, 0, (size_t)MF * sizeof(gfs_file), h->priv));
+  CK(cudaMemsetAsync(c.paths, 0, (size_t)MF * GFS_MAX_PATH, h->priv));
+  CK(cudaMemsetAsync(c.cpl, 0, (size_t)R * 8, h->priv));
+  CK(cudaMemsetAsync(c.ack, 0, (size_t)R * 8, h->priv));
+  CK(cudaMemsetAsync(c.ring_tail, 0, 8, h->priv));
+  CK(cudaMemsetAsync(c.ctr, 0, ctr_bytes, h->priv));
+  {
+    int ir = gfs_internal_init_metadata(&c, h->priv);
+    if (ir) {
+      rc = ir;
+      goto fail;
+    }
+  }
+  CK(cudaMalloc((void**)&h->d, sizeof(gfs_ctx)));
+  CK(cudaMemcpyAsync(h->d, &c, sizeof(gfs_ctx), cudaMemcpyHostToDevice, h->priv));
+  CK(cudaStreamSynchronize(h->priv));
+
+  // stream write-value-64 for completions (CUDA 12: attribute 122)
+  {
+    void* fn = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    if (!(cfg->flags & GFS_F_NO_DMA_COMPLETION) &&
+        cudaGetDriverEntryPoint("cuStreamWriteValue64", &fn, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess && fn) {
+      void* fa = nullptr;
+      int ok = 0;
+      if (cudaGetDriverEntryPoint("cuDeviceGetAttribute", &fa, cudaEnableDefault, &q) == cudaSuccess && fa) {
+        CUdevice dev = cfg->device;
+        ((PFN_devAttr)fa)(&ok, (CUdevice_attribute)122 /* CAN_USE_64_BIT_STREAM_MEM_OPS */, dev);
+      }
+      if (ok) h->wv64 = (PFN_writeValue64)fn;
+    }
+  }
+
+  h->staging_bytes = cfg->page_size;
+  h->workers.resize(cfg->daemon_threads);
+  for (auto& w : h->workers) {
+    CK(cudaStreamCreateWithFlags(&w.stream, cudaStreamNonBlocking));
+    for (int b = 0; b < 2; ++b) {
+      CK(cudaHostAlloc((void**)&w.staging[b], h->staging_bytes, cudaHostAllocPortable));
+      CK(cudaEventCreateWithFlags(&w.ev[b], cudaEventDisableTiming));
+    }
+  }
+  if (!h->vt.open()) fprintf(stderr, "gpufs: version table unavailable; close-to-open checks use size/mtime only\n");
+  *out = h;
+  return 0;
+fail:
+  free_all(h);
+  delete h;
+  return rc ? rc : -EIO;
+}
+
+GFS_API int gfs_daemon(gfs_handle* h, int mode) {
+  if (!h) return -EINVAL;
+  if (!h->running.exchange(true)) {
+    for (size_t i = 0; i < h->workers.size(); ++i) h->workers[i].th = std::thread(worker_loop, h, (int)i);
+  }
+  if (mode == GFS_DAEMON_RUN) {
+    while (h->running.load()) usleep(1000);
+  }
+  return 0;
+}
+
+GFS_API int gfs_daemon_stop(gfs_handle* h) {
+  if (!h) return -EINVAL;
+  h->running.store(false);
+  for (auto& w : h->workers)
+    if (w.th.joinable()) w.th.join();
+  // tickets claimed by idle workers are handed out again on restart
+  // (the GPU's tail never passed them); resynchronise with the device tail.
+  unsigned long long tail = 0;
+  cudaMemcpyAsync(&tail, h->h.ring_tail, 8, cudaMemcpyDeviceToHost, h->priv);
+  cudaStreamSynchronize(h->priv);
+  h->next_ticket.store(tail);
+  return 0;
+}
+
+GFS_API int gfs_shutdown(gfs_handle* h) {
+  if (!h) return -EINVAL;
+  gfs_daemon_stop(h);
+  cudaSetDevice(h->cfg.device);
+  cudaStreamSynchronize(h->priv);
+  free_all(h);
+  delete h;
+  return 0;
+}
+
+GFS_API const gfs_ctx* gfs_device_ctx(gfs_handle* h) { return h ? h->d : nullptr; }
+
+GFS_API int gfs_stats(gfs_handle* h, uint64_t* out, int n, int reset) {
+  if (!h || !out) return -EINVAL;
+  std::vector<unsigned long long> buf((size_t)GFS_C_NCOUNTERS * GFS_CTR_SHARDS);
+  cudaSetDevice(h->cfg.device);
+  if (cudaMemcpyAsync(buf.data(), h->h.ctr, buf.size() * 8, cudaMemcpyDeviceToHost, h->priv) != cudaSuccess)
+    return -EIO;
+  if (cudaStreamSynchronize(h->priv) != cudaSuccess) return -EIO;
+  for (int i = 0; i < n && i < GFS_C_NCOUNTERS; ++i) {
+    uint64_t s = 0;
+    for (int k = 0; k < GFS_CTR_SHARDS; ++k) s += buf[(size_t)i * GFS_CTR_SHARDS + k];
+    out[i] = s;
+  }
+  if (reset) {
+    cudaMemsetAsync(h->h.ctr, 0, buf.size() * 8, h->priv);
+    cudaStreamSynchronize(h->priv);
+  }
+  return GFS_C_NCOUNTERS;
+}
+
+GFS_API int gfs_host_stats(gfs_handle* h, uint64_t* out, int n) {
+  if (!h || !out) return -EINVAL;
+  for (int i = 0; i < n && i < HS_N; ++i) out[i] = h->hs[i].load();
+  return HS_N;
+}
+
+GFS_API int gfs_info(gfs_handle* h, uint64_t* out, int n) {
+  if (!h || !out) return -EINVAL;
+  uint64_t v[7] = {h->h.page_size, h->h.nframes, h->h.max_files, h->h.max_nodes, h->h.ring_slots,
+                   h->workers.size(), h->wv64 ? 1u : 0u};
+  for (int i = 0; i < n && i < 7; ++i) out[i] = v[i];
+  return 7;
+}

@@ -1,0 +1,336 @@
+// gfs_kernels.cu — kernels built on the device API (gpufs_device.cuh) and the
+// extern "C" launchers declared in include/gpufs.h.
+//
+//   k_init_metadata   pframe/counter initialisation at gfs_init
+//   k_gread_calls     parity harness: per-block gopen + gread/gmmap calls
+//   k_seqread         C2 / K1 sequential sweep + position checksum
+//   k_randread        K4 cache-hit reads into shared memory and
+//                     its raw-memory baseline with the same access pattern
+//   k_gwrite_calls    gwrite harness (O_GWRONCE)
+//   k_fileop          gfsync / gftruncate / gfstat / gopen+gclose
+#include <cuda_runtime.h>
+#include <errno.h>
+#include <stdint.h>
+#include <string.h>
+
+#include "gpufs.h"
+#include "gpufs_device.cuh"
+
+#define GFS_API extern "C" __attribute__((visibility("default")))
+
+using namespace gfs;
+
+namespace {
+
+__global__ void k_init_metadata(gfs_ctx c) {
+  const size_t stride = (size_t)gridDim.x * blockDim.x;
+  for (size_t i = blockIdx.x * (size_t)blockDim.x + threadIdx.x; i < c.nframes; i += stride) {
+    c.f_state[i] = GFS_ST_EVICTING;  // never-used frames are handed out by fresh_next only
+    c.f_tag[i] = GFS_TAG_NONE;
+    c.f_file[i] = 0xFFFFFFFFu;
+    c.f_valid[i] = 0;
+    c.f_lo[i] = GFS_DIRTY_NONE;
+    c.f_hi[i] = 0;
+    c.f_written[i] = 0;
+    c.f_stamp[i] = 0;
+  }
+  if (blockIdx.x == 0 && threadIdx.x == 0) {
+    *c.fresh_next = 0;
+    *c.hand = 0;
+    *c.node_next = 1;  // node 0 is the null node
+    *c.node_free_top = 0;
+    *c.node_lock = 0;
+    *c.uid_next = 1;
+  }
+}
+
+// Position-weighted checksum of `n` bytes at `p` holding file bytes starting at
+// file offset `foff` (8-byte aligned): sum_j w_j * (2j + 1), j global word index.
+__device__ __forceinline__ uint64_t checksum_words(const uint8_t* p, uint64_t foff, uint64_t n, int tid,
+                                                   int nthr, bool cg) {
+  uint64_t s = 0;
+  const uint64_t j0 = foff >> 3;
+  const uint64_t nw = n >> 3;
+  if (((uintptr_t)p & 15) == 0) {
+    const uint64_t nv = nw >> 1;
+    const ulonglong2* p2 = (const ulonglong2*)p;
+    for (uint64_t i = tid; i < nv; i += nthr) {
+      ulonglong2 v = cg ? __ldcg(p2 + i) : p2[i];
+      const uint64_t j = j0 + 2 * i;
+      s += v.x * (2 * j + 1) + v.y * (2 * j + 3);
+    }
+    if ((nw & 1) && tid == 0) {
+      const uint64_t* p1 = (const uint64_t*)p;
+      s += (cg ? __ldcg(p1 + nw - 1) : p1[nw - 1]) * (2 * (j0 + nw - 1) + 1);
+    }
+  } else {
+    for (uint64_t i = tid; i < nw; i += nthr) {
+      uint64_t v = 0;
+      for (int b = 0; b < 8; ++b) v |= (uint64_t)p[8 * i + b] << (8 * b);
+      s += v * (2 * (j0 + i) + 1);
+    }
+  }
+  if (tid == 0 && (n & 7)) {  // ragged tail: missing bytes count as zero
+    uint64_t v = 0;
+    for (uint64_t b = 0; b < (n & 7); ++b) v |= (uint64_t)p[8 * nw + b] << (8 * b);
+    s += v * (2 * (j0 + nw) + 1);
+  }
+  return s;
+}
+
+__device__ __forceinline__ uint64_t warp_sum(uint64_t v) {
+  for (int o = 16; o; o >>= 1) v += __shfl_xor_sync(0xFFFFFFFFu, v, o);
+  return v;
+}
+
+__device__ __forceinline__ void note_err(int64_t* d_err, int64_t r) {
+  if (r < 0 && d_err) atomicMin((long long*)d_err, (long long)r);
+}
+
+__global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint32_t ncalls, const uint64_t* off,
+                              const uint64_t* len, const uint64_t* dstoff, uint8_t* dst, int64_t* ret,
+                              uint32_t smem_bytes) {
+  extern __shared__ __align__(16) uint8_t smem[];
+  const int tid = threadIdx.x;
+  const int fd = gopen(c, path, GFS_O_RDONLY);
+  for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
+    int64_t r;
+    if (fd < 0) {
+      r = fd;
+    } else if (mode == 0) {
+      r = gread(c, fd, off[i], len[i], dst + dstoff[i]);
+    } else if (mode == 1) {
+      uint64_t m = 0;
+      uint8_t* p = (uint8_t*)gmmap(c, nullptr, len[i], 0, 0, fd, off[i], &m);
+      if (p) {
+        // user copy out of the mapped page (frames are read with .cg loads)
+        detail::block_copy_from_frame(dst + dstoff[i], p, m, tid, blockDim.x);
+        __syncthreads();
+        gmunmap(c, p, m);
+        r = (int64_t)m;
+      } else {
+        r = 0;
+      }
+    } else if (len[i] > smem_bytes) {
+      r = -EINVAL;  // destination would overflow the shared buffer
+    } else {
+      r = gread(c, fd, off[i], len[i], smem);
+      if (r > 0)
+        for (int64_t k = tid; k < r; k += blockDim.x) dst[dstoff[i] + k] = smem[k];
+      __syncthreads();
+    }
+    if (tid == 0) ret[i] = r;
+  }
+  if (fd >= 0) gclose(c, fd);
+}
+
+__global__ void k_seqread(const gfs_ctx* c, const char* path, uint64_t file_off, uint64_t total, uint64_t chunk,
+                          int use_mmap, uint8_t* scratch, uint64_t* sum, int64_t* err) {
+  const int tid = threadIdx.x, nthr = blockDim.x;
+  const int fd = gopen(c, path, GFS_O_RDONLY);
+  if (fd < 0) {
+    if (tid == 0) note_err(err, fd);
+    return;
+  }
+  const uint64_t nchunks = (total + chunk - 1) / chunk;
+  const uint64_t per = (nchunks + gridDim.x - 1) / gridDim.x;
+  const uint64_t c0 = blockIdx.x * per, c1 = c0 + per < nchunks ? c0 + per : nchunks;
+  uint64_t s = 0;
+  uint8_t* buf = scratch + (size_t)blockIdx.x * chunk;
+  for (uint64_t k = c0; k < c1; ++k) {
+    const uint64_t o = file_off + k * chunk;
+    const uint64_t want = (k + 1) * chunk <= total ? chunk : total - k * chunk;
+    if (!use_mmap) {
+      const int64_t r = gread(c, fd, o, want, buf);
+      if (r < 0) {
+        if (tid == 0) note_err(err, r);
+        break;
+      }
+      s += checksum_words(buf, o, (uint64_t)r, tid, nthr, false);
+    } else {
+      uint64_t done = 0;
+      while (done < want) {  // gmmap maps at most one page: loop over the prefix
+        uint64_t m = 0;
+        const uint8_t* p = (const uint8_t*)gmmap(c, nullptr, want - done, 0, 0, fd, o + done, &m);
+        if (!p || m == 0) {
+          if (tid == 0) note_err(err, -EIO);
+          break;
+        }
+        s += checksum_words(p, o + done, m, tid, nthr, true);
+        __syncthreads();
+        gmunmap(c, (void*)p, m);
+        done += m;
+      }
+    }
+  }
+  s = warp_sum(s);
+  if ((tid & 31) == 0) atomicAdd((unsigned long long*)sum, (unsigned long long)s);
+  gclose(c, fd);
+}
+
+__global__ void k_randread(const gfs_ctx* c, const char* path, int raw, const uint8_t* rawp, uint32_t chunk,
+                           uint32_t calls, const uint64_t* offs, uint64_t* sum, int64_t* err) {
+  extern __shared__ __align__(16) uint8_t smem[];
+  const int tid = threadIdx.x, nthr = blockDim.x;
+  int fd = 0;
+  if (!raw) {
+    fd = gopen(c, path, GFS_O_RDONLY);
+    if (fd < 0) {
+      if (tid == 0) note_err(err, fd);
+      return;
+    }
+  }
+  uint64_t s = 0;
+  const uint64_t* my = offs + (size_t)blockIdx.x * calls;
+  for (uint32_t i = 0; i < calls; ++i) {
+    const uint64_t o = my[i];
+    int64_t r;
+    if (raw) {
+      __syncthreads();
+      detail::block_copy_from_frame(smem, rawp + o, chunk, tid, nthr);
+      __syncthreads();
+      r = chunk;
+    } else {
+      r = gread(c, fd, o, chunk, smem);
+      if (r < 0) {
+        if (tid == 0) note_err(err, r);
+        break;
+      }
+    }
+    s += checksum_words(smem, o, (uint64_t)r, tid, nthr, false);
+  }
+  s = warp_sum(s);
+  if ((tid & 31) == 0) atomicAdd((unsigned long long*)sum, (unsigned long long)s);
+  if (!raw) gclose(c, fd);
+}
+
+__global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
+                               const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret) {
+  const int fd = gopen(c, path, GFS_O_GWRONCE);
+  for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
+    int64_t r = fd < 0 ? fd : gwrite(c, fd, off[i], len[i], src + srcoff[i]);
+    if (threadIdx.x == 0) ret[i] = r;
+  }
+  if (fd >= 0) gclose(c, fd);
+}
+
+__global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, uint64_t arg, int64_t* ret) {
+  const int fd = gopen(c, path, flags);
+  int64_t r = fd;
+  if (fd >= 0) {
+    if (op == 0) r = gfsync(c, fd);
+    else if (op == 1) r = gftruncate(c, fd, arg);
+    else if (op == 2) r = gfstat_size(c, fd);
+    else r = fd;
+    const int cr = gclose(c, fd);
+    if (r >= 0 && cr < 0) r = cr;
+  }
+  if (threadIdx.x == 0) *ret = r;
+}
+
+int launch_err(cudaError_t e) { return e == cudaSuccess ? 0 : -EIO; }
+
+// Stage a host path string in device memory, ordered on `s`. The staging
+// buffer is a small per-process ring of pinned+device buffers.
+struct PathStage {
+  char* d = nullptr;
+  char* h = nullptr;
+  cudaEvent_t ev[64];
+  bool used[64];
+  int next = 0;
+  bool init = false;
+};
+PathStage g_ps;
+
+const char* stage_path(const char* path, cudaStream_t s) {
+  if (!path) return nullptr;
+  const size_t n = strlen(path);
+  if (n >= GFS_MAX_PATH) return nullptr;
+  if (!g_ps.init) {
+    if (cudaMalloc((void**)&g_ps.d, 64 * GFS_MAX_PATH) != cudaSuccess) return nullptr;
+    if (cudaHostAlloc((void**)&g_ps.h, 64 * GFS_MAX_PATH, cudaHostAllocPortable) != cudaSuccess) return nullptr;
+    for (int i = 0; i < 64; ++i) {
+      cudaEventCreateWithFlags(&g_ps.ev[i], cudaEventDisableTiming);
+      g_ps.used[i] = false;
+    }
+    g_ps.init = true;
+  }
+  const int k = g_ps.next;
+  g_ps.next = (k + 1) % 64;
+  if (g_ps.used[k]) cudaEventSynchronize(g_ps.ev[k]);
+  memcpy(g_ps.h + (size_t)k * GFS_MAX_PATH, path, n + 1);
+  if (cudaMemcpyAsync(g_ps.d + (size_t)k * GFS_MAX_PATH, g_ps.h + (size_t)k * GFS_MAX_PATH, n + 1,
+                      cudaMemcpyHostToDevice, s) != cudaSuccess)
+    return nullptr;
+  cudaEventRecord(g_ps.ev[k], s);
+  g_ps.used[k] = true;
+  return g_ps.d + (size_t)k * GFS_MAX_PATH;
+}
+
+}  // namespace
+
+extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s) {
+  k_init_metadata<<<1024, 256, 0, s>>>(*hctx);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
+                          const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
+                          int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes) {
+  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || mode > 2) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = stage_path(path, s);
+  if (!dp) return -ENAMETOOLONG;
+  if (mode == 2 && smem_bytes > 48 * 1024)
+    cudaFuncSetAttribute(k_gread_calls, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem_bytes);
+  k_gread_calls<<<grid, block, mode == 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,
+                                                                d_dstoff, d_dst, d_ret, smem_bytes);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint64_t file_off, uint64_t total,
+                            uint64_t chunk, int use_mmap, uint8_t* d_scratch, uint64_t* d_sum, int64_t* d_err,
+                            uint32_t grid, uint32_t block) {
+  if (!h || grid == 0 || block == 0 || block > 1024 || chunk == 0 || (chunk & 7) || (file_off & 7)) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = stage_path(path, s);
+  if (!dp) return -ENAMETOOLONG;
+  k_seqread<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, file_off, total, chunk, use_mmap, d_scratch, d_sum, d_err);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
+                             uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
+                             int64_t* d_err, uint32_t grid, uint32_t block) {
+  if ((!raw && !h) || (raw && !d_raw) || grid == 0 || block == 0 || chunk == 0 || (chunk & 15) ||
+      chunk > 200 * 1024)
+    return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = raw ? nullptr : stage_path(path, s);
+  if (!raw && !dp) return -ENAMETOOLONG;
+  if (chunk > 48 * 1024) cudaFuncSetAttribute(k_randread, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
+  k_randread<<<grid, block, chunk, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
+                                        d_off, d_sum, d_err);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncalls, const uint64_t* d_off,
+                           const uint64_t* d_len, const uint64_t* d_srcoff, const uint8_t* d_src, int64_t* d_ret,
+                           uint32_t grid, uint32_t block) {
+  if (!h || grid == 0 || block == 0 || block > 1024) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = stage_path(path, s);
+  if (!dp) return -ENAMETOOLONG;
+  k_gwrite_calls<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int flags, int op, uint64_t arg,
+                           int64_t* d_ret) {
+  if (!h || !d_ret) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = stage_path(path, s);
+  if (!dp) return -ENAMETOOLONG;
+  k_fileop<<<1, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, op, arg, d_ret);
+  return launch_err(cudaGetLastError());
+}

@@ -1,0 +1,162 @@
+"""GPU parity: gread / gmmap through the C ABI vs the oracle (bit-exact).
+
+Inputs: seeded splitmix files and seeded (off, len) call lists from gen/.
+Expected values: oracle.pread (the plain pread definition) per call, and
+oracle.checksum for sweeps. Runs on a B200 via gpurun.
+"""
+import os
+
+import numpy as np
+import pytest
+
+import gen
+import oracle
+
+pytestmark = [pytest.mark.gpu, pytest.mark.timeout(600)]
+
+
+@pytest.fixture(scope="module")
+def g():
+    import paper_conf_asplos_silbersteinfkw13_b200 as g
+    g.build.build()
+    return g
+
+
+def _fs(g, **kw):
+    kw.setdefault("timeout_ms", 30000)
+    kw.setdefault("daemon_threads", 4)
+    return g.GpuFS(**kw)
+
+
+def check_calls(path, size, offs, lens, ret, dst, dstoff):
+    for i, (o, l) in enumerate(zip(offs.tolist(), lens.tolist())):
+        exp = oracle.pread(path, size, o, l)
+        assert ret[i] == len(exp), (i, o, l, ret[i])
+        got = dst[int(dstoff[i]):int(dstoff[i]) + len(exp)].tobytes()
+        assert got == exp, (i, o, l)
+
+
+@pytest.mark.parametrize("P,cache_pages,batch,grid", [
+    (4096, 4096, 32, 64),      # cache larger than file: misses then hits
+    (4096, 64, 1, 16),         # tiny cache: heavy miss/evict/refetch churn
+    (65536, 32, 2, 8),
+    (1 << 21, 8, 1, 4),        # 2 MiB pages, 16 MiB cache < file
+])
+def test_gread_random_calls(g, shmdir, P, cache_pages, batch, grid):
+    size = 3 * (1 << 21) + 12345 if P >= 65536 else 40 * 4096 * 16 + 77
+    path = gen.splitmix_file(os.path.join(shmdir, "f.bin"), size, seed=5)
+    offs, lens = gen.random_calls(17, 600, size, max(3 * P // 2, 20000), page_size=P)
+    with _fs(g, cache_bytes=cache_pages * P, page_size=P, max_batch=batch) as fs:
+        for rep in range(2):
+            ret, dst, dstoff = fs.gread_calls(path, offs, lens, mode=0, grid=grid)
+            check_calls(path, size, offs, lens, ret, dst, dstoff)
+        st = fs.stats()
+        assert st["timeout"] == 0 and st["enomem"] == 0
+        assert st["miss"] > 0
+        if cache_pages * P > size:
+            assert st["evict"] == 0
+
+
+def test_gread_hits_after_warm(g, shmdir):
+    P = 65536
+    size = 200 * P + 5
+    path = gen.splitmix_file(os.path.join(shmdir, "w.bin"), size, seed=8)
+    with _fs(g, cache_bytes=512 * P, page_size=P) as fs:
+        fs.gread_calls(path, [0], [size], grid=1)
+        st0 = fs.stats()
+        assert st0["miss"] == 201  # one miss per page of the file (O1 invariant)
+        offs, lens = gen.random_calls(3, 500, size, 3 * P, page_size=P)
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, grid=64)
+        check_calls(path, size, offs, lens, ret, dst, dstoff)
+        st1 = fs.stats()
+        assert st1["miss"] == st0["miss"] and st1["hit"] > st0["hit"]
+
+
+def test_gmmap_prefix(g, shmdir):
+    P = 16384
+    size = 50 * P + 999
+    path = gen.splitmix_file(os.path.join(shmdir, "m.bin"), size, seed=9)
+    offs, lens = gen.random_calls(4, 400, size, 3 * P, page_size=P)
+    with _fs(g, cache_bytes=16 * P, page_size=P, max_batch=1) as fs:
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, mode=1, grid=8)
+    for i, (o, l) in enumerate(zip(offs.tolist(), lens.tolist())):
+        m = 0 if (o >= size or l == 0) else min(l, P - o % P, size - o)
+        assert ret[i] == m, (o, l, ret[i], m)
+        assert dst[int(dstoff[i]):int(dstoff[i]) + m].tobytes() == oracle.pread(path, size, o, m)
+
+
+def test_gread_into_shared_memory(g, shmdir):
+    P = 65536
+    size = 64 * P
+    path = gen.splitmix_file(os.path.join(shmdir, "s.bin"), size, seed=10)
+    offs, lens = gen.random_calls(5, 300, size, 32768, page_size=P)
+    lens[0] = 40000  # larger than the shared buffer: rejected, nothing written
+    with _fs(g, cache_bytes=128 * P, page_size=P) as fs:
+        ret, dst, dstoff = fs.gread_calls(path, offs, np.minimum(lens, 40000), mode=2, grid=32, smem=32768)
+    assert ret[0] == -22
+    ok = np.minimum(lens, 40000) <= 32768
+    check_calls(path, size, offs[ok], lens[ok], ret[ok], dst, dstoff[ok])
+
+
+@pytest.mark.parametrize("locked", [0, 1])
+def test_locked_traversal_same_bytes(g, shmdir, locked):
+    P = 4096
+    size = 300 * P + 1
+    path = gen.splitmix_file(os.path.join(shmdir, "l.bin"), size, seed=12)
+    offs, lens = gen.random_calls(6, 400, size, 5 * P, page_size=P)
+    with _fs(g, cache_bytes=1024 * P, page_size=P, flags=locked) as fs:
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, grid=48)
+        st = fs.stats()
+    check_calls(path, size, offs, lens, ret, dst, dstoff)
+    if locked:
+        assert st["locked"] > 0 and st["lockfree"] == 0
+    else:
+        assert st["lockfree"] > 0
+
+
+@pytest.mark.parametrize("P,cache_mb,use_mmap", [(1 << 21, 8, 0), (65536, 4, 0), (1 << 21, 8, 1)])
+def test_seqread_sweep_larger_than_cache(g, shmdir, P, cache_mb, use_mmap):
+    size = 64 << 20
+    path = gen.splitmix_file(os.path.join(shmdir, "seq.bin"), size, seed=21)
+    grid = 4 if P == 1 << 21 else 16
+    with _fs(g, cache_bytes=cache_mb << 20, page_size=P, max_batch=1) as fs:
+        s, err = fs.seqread(path, size, P, use_mmap=bool(use_mmap), grid=grid)
+        st = fs.stats()
+    assert err == 0
+    assert s == oracle.checksum(path, 0, size)
+    npages = size // P
+    assert st["miss"] == npages and st["evict"] == npages - (cache_mb << 20) // P
+
+
+def test_randread_smem_checksum(g, shmdir):
+    P = 1 << 17
+    size = 256 * P
+    chunk = 16384
+    path = gen.splitmix_file(os.path.join(shmdir, "k4.bin"), size, seed=31)
+    grid, calls = 64, 50
+    rng = np.random.default_rng(0)
+    offs = (rng.integers(0, size // chunk, size=grid * calls) * chunk).astype(np.uint64)
+    expect = sum(oracle.checksum(path, int(o), chunk) for o in offs) % (1 << 64)
+    with _fs(g, cache_bytes=512 * P, page_size=P) as fs:
+        s, err = fs.randread(path, chunk, offs, grid)
+        assert err == 0 and s == expect
+        s2, err2 = fs.randread(path, chunk, offs, grid)
+        st = fs.stats()
+        assert err2 == 0 and s2 == expect
+        import torch
+        raw = torch.as_tensor(np.fromfile(path, dtype=np.uint8), device="cuda")
+        s3, _ = fs.randread(None, chunk, offs, grid, raw=raw)
+        assert s3 == expect
+    assert st["miss"] <= 256
+
+
+def test_errors(g, shmdir):
+    with _fs(g, cache_bytes=64 << 20, page_size=65536) as fs:
+        ret, _, _ = fs.gread_calls(os.path.join(shmdir, "missing.bin"), [0], [10], grid=1)
+        assert ret[0] == -2  # -ENOENT from the host open
+        assert fs.gfstat(os.path.join(shmdir, "missing.bin")) == -2
+        p = os.path.join(shmdir, "x.bin")
+        gen.splitmix_file(p, 1000, 1)
+        assert fs.gfstat(p) == 1000
+        ret, _, _ = fs.gread_calls(p, [0, 999, 1000, 5000], [2000, 10, 1, 1], grid=2)
+        assert ret.tolist() == [1000, 1, 0, 0]
