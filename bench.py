@@ -1,0 +1,376 @@
+#!/usr/bin/env python
+"""bench.py — GPUfs buffer-cache read path on B200 (BASELINE.json configs[1]).
+
+Headline workload (N=1, configs[1]): sequential gread sweep over one file
+larger than the 4 GiB GPU cache (P = 2 MiB), so every page is a miss RPC +
+pread + DMA fill + LRU eviction, followed by the block's checksum of the
+bytes read. value = file GB/s of the sweep kernel (CUDA events on its stream).
+
+Also measured in the same run (extra keys):
+  hit   — K4-shape cache-hit gread (16 KiB chunks -> shared memory at random
+          offsets of a pre-warmed file), against HBM and against a raw-memory
+          baseline kernel with the same access pattern;
+  grep  — (when available) grep -w corpus GB/s.
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+Multi-GPU: one process per GPU (torchrun), each rank sweeps its own file with
+a private cache (weak scaling); the only collective is the final all-reduce of
+checksums. Timing = max over ranks of the device-timed region.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+MEASURED = os.path.join(ROOT, "MEASURED_PEAKS.json")
+FALLBACK_HBM = 6650.0
+
+
+def peaks():
+    try:
+        with open(MEASURED) as f:
+            d = json.load(f)
+        return float(d["hbm_gbs"]), "measured"
+    except Exception:
+        return FALLBACK_HBM, "fallback"
+
+
+class Clocks:
+    """Sample nvidia-smi clocks and throttle reasons during the timed region."""
+
+    def __init__(self, index: int):
+        self.index = index
+        self.samples = []
+        self._stop = threading.Event()
+        self._th = None
+
+    def __enter__(self):
+        def run():
+            q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,"
+                 "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+                 "clocks_event_reasons.sw_power_cap")
+            while not self._stop.is_set():
+                try:
+                    out = subprocess.run(["nvidia-smi", "-i", str(self.index), f"--query-gpu={q}",
+                                          "--format=csv,noheader,nounits"], capture_output=True, text=True,
+                                         timeout=5).stdout.strip()
+                    if out:
+                        self.samples.append([x.strip() for x in out.split(",")])
+                except Exception:
+                    pass
+                self._stop.wait(0.2)
+
+        self._th = threading.Thread(target=run, daemon=True)
+        self._th.start()
+        return self
+
+    def __exit__(self, *a):
+        self._stop.set()
+        if self._th:
+            self._th.join(timeout=10)
+
+    def summary(self):
+        if not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"]}
+        sm = [float(s[0]) for s in self.samples if s[0].replace(".", "").isdigit()]
+        mx = [float(s[1]) for s in self.samples if s[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for s in self.samples for i in range(4) if len(s) > i + 2 and
+                          s[i + 2].strip().lower() == "active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.samples)}
+
+
+def pinned_h2d_gbs(torch, dev, nbytes=256 << 20, reps=10):
+    """In-run pinned host->device cudaMemcpyAsync bandwidth (the miss-fill roofline)."""
+    h = torch.empty(nbytes, dtype=torch.uint8).pin_memory()
+    d = torch.empty(nbytes, dtype=torch.uint8, device=dev)
+    s = torch.cuda.Stream(device=dev)
+    best = 0.0
+    for _ in range(reps):
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        with torch.cuda.stream(s):
+            e0.record(s)
+            d.copy_(h, non_blocking=True)
+            e1.record(s)
+        s.synchronize()
+        best = max(best, nbytes / (e0.elapsed_time(e1) * 1e-3) / 1e9)
+    del h, d
+    return best
+
+
+def dist_env():
+    ws = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return ws, rank, local
+
+
+# ---------------------------------------------------------------------- reference arm
+def run_reference(args):
+    """The CPU oracle as it stands (pread + position checksum), bounded sample."""
+    ws, rank, _ = dist_env()
+    if ws > 1 and rank != 0:
+        return
+    import gen
+    import oracle
+    size = args.file_gib << 30
+    path = gen.splitmix_file(f"/dev/shm/gfs_bench_c2_{size}_r0.bin", size, seed=1000)
+    sample = min(size, args.ref_sample_mib << 20)
+    oracle.checksum(path, 0, 1 << 20)  # warm
+    times = []
+    for i in range(args.warmup + args.steps):
+        off = ((i * 7919) % max(1, size // sample)) * sample
+        t0 = time.perf_counter()
+        oracle.checksum(path, off, sample)
+        dt = time.perf_counter() - t0
+        if i >= args.warmup:
+            times.append(dt)
+    ms = 1e3 * statistics.mean(times)
+    val = sample / (ms * 1e-3) / 1e9
+    line = {"impl": "reference", "metric": "gread GB/s (miss fill, sequential sweep > cache)", "value": round(val, 3),
+            "unit": "GB/s", "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+            "ms_per_step": round(ms, 3), "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+            "dtype": "u8", "data": "synthetic",
+            "config": {"workload": f"C2 sequential sweep, {args.file_gib} GiB file, oracle pread+checksum sample "
+                                   f"{args.ref_sample_mib} MiB per step"},
+            "cpu_baseline": {"value": round(val, 3), "unit": "GB/s", "cores": 1, "kind": "oracle",
+                             "sample": f"{args.ref_sample_mib} MiB of the {args.file_gib} GiB file per step"},
+            "e2e": {"value": round(val, 3), "unit": "GB/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ---------------------------------------------------------------------- our arm
+def run_ours(args):
+    import torch
+    import torch.distributed as dist
+
+    import gen
+    import paper_conf_asplos_silbersteinfkw13_b200 as g
+
+    ws, rank, local = dist_env()
+    if ws > 1:
+        dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
+    torch.cuda.set_device(local)
+    dev = f"cuda:{local}"
+    g.build.build()
+    hbm, hbm_src = peaks()
+
+    size = args.file_gib << 30
+    P = args.page_kib << 10
+    path = gen.splitmix_file(f"/dev/shm/gfs_bench_c2_{size}_r{rank}.bin", size, seed=1000 + rank)
+    h2d = pinned_h2d_gbs(torch, dev)
+
+    fs = g.GpuFS(cache_bytes=args.cache_gib << 30, page_size=P, device=local, daemon_threads=args.daemon_threads,
+                 max_batch=1, timeout_ms=args.timeout_ms)
+    grid = args.grid
+    stream = torch.cuda.Stream(device=dev)
+    scratch = torch.empty(grid * P, dtype=torch.uint8, device=dev)
+    out = torch.zeros(2, dtype=torch.int64, device=dev)
+
+    def step():
+        out.zero_()
+        fs.seqread(path, size, P, grid=grid, stream=stream, sync=False, scratch=scratch, out=out)
+
+    with torch.cuda.stream(stream):
+        for _ in range(args.warmup):
+            step()
+        stream.synchronize()
+        v = out.cpu().numpy()
+        if v[1] != 0:
+            print("stats", fs.stats(), fs.host_stats(), fs.info(), file=sys.stderr)
+            raise SystemExit(f"gread sweep error {v[1]}")
+        fs.stats(reset=True)
+        if ws > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+        evs = []
+        with Clocks(local) as clk:
+            for _ in range(args.steps):
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                e0.record(stream)
+                step()
+                e1.record(stream)
+                evs.append((e0, e1))
+            stream.synchronize()
+        torch.cuda.synchronize()
+    step_ms = [a.elapsed_time(b) for a, b in evs]
+    ms = float(np.mean(step_ms))
+    st = fs.stats()
+    hst = fs.host_stats()
+    checksum = int(out[0].item()) & ((1 << 64) - 1)
+
+    # e2e: the public API call with host-side result read, wall clock, inputs from tmpfs
+    # NOTE: never issue a synchronous copy (tensor.cpu()) while a GPUfs kernel
+    # runs: it can hold driver locks the daemon's async DMA needs. Wait on the
+    # stream first, then read the result into pinned memory.
+    res = torch.empty(2, dtype=torch.int64).pin_memory()
+    torch.cuda.synchronize()
+    t0 = time.perf_counter()
+    with torch.cuda.stream(stream):
+        for _ in range(args.steps):
+            step()
+            stream.synchronize()
+            res.copy_(out, non_blocking=True)  # D2H of the step's result (checksum, error)
+            stream.synchronize()
+    e2e_s = (time.perf_counter() - t0) / args.steps
+    if int(res[1]) != 0:
+        raise SystemExit(f"gread sweep error {int(res[1])}")
+
+    # cache-hit phase (K4 shape): pre-warm a file that fits, random 16 KiB greads into smem
+    hit = None
+    if not args.no_hit:
+        hit = hit_phase(args, torch, g, gen, fs, dev, stream, hbm, rank)
+
+    tmax = torch.tensor([ms], device=dev)
+    if ws > 1:
+        dist.all_reduce(tmax, op=dist.ReduceOp.MAX)
+        cs = torch.tensor([checksum & 0x7FFFFFFFFFFFFFFF], device=dev)
+        dist.all_reduce(cs)  # the final reduction (NCCL)
+    ms_max = float(tmax.item())
+    value = ws * size / (ms_max * 1e-3) / 1e9
+    achieved = size / (ms * 1e-3) / 1e9
+    clk_s = clk.summary()
+    fs.close()
+    if rank != 0:
+        return
+    line = {
+        "metric": "gread GB/s (miss fill, sequential sweep > cache)",
+        "value": round(value, 3), "unit": "GB/s", "n_gpus": ws, "steps": args.steps, "warmup": args.warmup,
+        "ms_per_step": round(ms_max, 3), "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+        "dtype": "u8", "data": "synthetic",
+        "config": {"workload": f"C2: sequential gread sweep of a {args.file_gib} GiB splitmix file per GPU, "
+                               f"{args.cache_gib} GiB GPU cache, {args.page_kib} KiB pages, grid {grid}x256, "
+                               f"{args.daemon_threads} daemon threads; tmpfs; file > cache and > L2 (no flush needed)",
+                   "page_kib": args.page_kib, "cache_gib": args.cache_gib, "file_gib": args.file_gib},
+        "roofline": {"bound": "h2d", "achieved": round(achieved, 3), "peak": round(h2d, 3), "unit": "GB/s",
+                     "frac": round(achieved / h2d, 4), "traffic": None,
+                     "peak_source": "pinned cudaMemcpyAsync H2D 256 MiB, best of 10, measured in this run"},
+        "e2e": {"value": round(size * ws / e2e_s / 1e9, 3), "unit": "GB/s", "h2d_bytes_per_step": size,
+                "d2h_bytes_per_step": 16},
+        "gpu_launches": args.steps,
+        "clocks": clk_s,
+        "counters": {k: st[k] for k in ("miss", "hit", "evict", "rpc", "timeout", "enomem", "ring_wait")},
+        "host": {"pread_GBps_per_thread": round(hst["bytes_h2d"] / max(hst["pread_ns"], 1), 3) if hst["pread_ns"] else None},
+        "checksum": hex(checksum),
+    }
+    if hit:
+        line["hit"] = hit
+    if not args.no_cpu:
+        line["cpu_baseline"] = cpu_baseline(args, path, size)
+    print(json.dumps(line), flush=True)
+
+
+def hit_phase(args, torch, g, gen, fs_unused, dev, stream, hbm, rank):
+    """K4: 16 KiB greads into shared memory at random offsets of a warm file."""
+    P = args.hit_page_kib << 10
+    size = args.hit_file_gib << 30
+    path = gen.splitmix_file(f"/dev/shm/gfs_bench_hit_{size}_r{rank}.bin", size, seed=2000 + rank)
+    chunk = 16384
+    grid = args.hit_grid
+    calls = args.hit_calls
+    rng = np.random.default_rng(7)
+    offs = (rng.integers(0, size // chunk, size=grid * calls) * chunk).astype(np.uint64)
+    d_off = torch.as_tensor(offs.view(np.int64), device=dev)
+    with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, device=torch.cuda.current_device(),
+                 daemon_threads=args.daemon_threads, timeout_ms=args.timeout_ms) as fs:
+        s, err = fs.seqread(path, size, P, grid=296)  # pre-warm
+        assert err == 0
+        fs.stats(reset=True)
+        out = torch.zeros(2, dtype=torch.int64, device=dev)
+        raw = torch.empty(size, dtype=torch.uint8, device=dev)
+        raw.copy_(torch.from_file(path, shared=False, size=size, dtype=torch.uint8), non_blocking=False)
+
+        def timed(fn, reps):
+            ts = []
+            for _ in range(reps):
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                e0.record(stream)
+                fn()
+                e1.record(stream)
+                stream.synchronize()
+                ts.append(e0.elapsed_time(e1))
+            return float(np.median(ts))
+
+        with torch.cuda.stream(stream):
+            run_g = lambda: fs.randread(path, chunk, d_off, grid, block=args.hit_block, stream=stream, sync=False,
+                                        out=out)
+            run_r = lambda: fs.randread(None, chunk, d_off, grid, block=args.hit_block, raw=raw, stream=stream,
+                                        sync=False, out=out)
+            for _ in range(2):
+                run_g()
+                run_r()
+            ms_g = timed(run_g, 5)
+            ms_r = timed(run_r, 5)
+            out.zero_()
+            run_g()
+            stream.synchronize()
+            sg = int(out[0].item()) & ((1 << 64) - 1)
+            out.zero_()
+            run_r()
+            stream.synchronize()
+            sr = int(out[0].item()) & ((1 << 64) - 1)
+        st = fs.stats()
+        del raw
+    nbytes = grid * calls * chunk
+    gbs = nbytes / (ms_g * 1e-3) / 1e9
+    return {"workload": f"K4: {grid} blocks x {calls} x 16 KiB gread -> smem, random offsets, {args.hit_file_gib} GiB "
+                        f"warm file, {args.hit_page_kib} KiB pages",
+            "GBps": round(gbs, 3), "raw_GBps": round(nbytes / (ms_r * 1e-3) / 1e9, 3),
+            "vs_raw": round(ms_r / ms_g, 4),
+            "roofline": {"bound": "hbm", "achieved": round(gbs, 3), "peak": hbm, "unit": "GB/s",
+                         "frac": round(gbs / hbm, 4), "traffic": None,
+                         "note": "1 algorithmic HBM byte per delivered byte (frame read; destination is smem)"},
+            "checksum_match_raw": sg == sr, "misses_after_warm": st["miss"], "ms": round(ms_g, 3)}
+
+
+def cpu_baseline(args, path, size):
+    import oracle
+    sample = min(size, args.ref_sample_mib << 20)
+    t0 = time.perf_counter()
+    oracle.checksum(path, 0, sample)
+    dt = time.perf_counter() - t0
+    return {"value": round(sample / dt / 1e9, 3), "unit": "GB/s", "cores": 1, "kind": "oracle",
+            "sample": f"oracle pread+checksum of the first {args.ref_sample_mib} MiB of the sweep file"}
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--file-gib", type=int, default=8)
+    ap.add_argument("--cache-gib", type=int, default=4)
+    ap.add_argument("--page-kib", type=int, default=2048)
+    ap.add_argument("--grid", type=int, default=296)
+    ap.add_argument("--daemon-threads", type=int, default=12)
+    ap.add_argument("--hit-file-gib", type=int, default=4)
+    ap.add_argument("--hit-page-kib", type=int, default=512)
+    ap.add_argument("--hit-grid", type=int, default=592)
+    ap.add_argument("--hit-block", type=int, default=256)
+    ap.add_argument("--hit-calls", type=int, default=2048)
+    ap.add_argument("--ref-sample-mib", type=int, default=2048)
+    ap.add_argument("--timeout-ms", type=int, default=60000)
+    ap.add_argument("--no-hit", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    args = ap.parse_args()
+    if args.impl == "reference":
+        run_reference(args)
+    else:
+        run_ours(args)
+
+
+if __name__ == "__main__":
+    main()

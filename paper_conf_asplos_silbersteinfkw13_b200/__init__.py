@@ -133,10 +133,10 @@ def gfs_host_stats(h: int) -> dict:
 
 
 def gfs_info(h: int) -> dict:
-    a = (ctypes.c_uint64 * 7)()
-    _ck(lib().gfs_info(h, a, 7), "gfs_info")
+    a = (ctypes.c_uint64 * 9)()
+    _ck(lib().gfs_info(h, a, 9), "gfs_info")
     return dict(zip(["page_size", "nframes", "max_files", "max_nodes", "ring_slots", "daemon_threads",
-                     "stream_write_value64"], (int(x) for x in a)))
+                     "stream_write_value64", "host_next_ticket", "device_ring_tail"], (int(x) for x in a)))
 
 
 # ------------------------------------------------------------------ launchers

@@ -123,10 +123,12 @@ class GpuFS:
     def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None):
         torch = _torch()
         dev = f"cuda:{self.device}"
-        offs = np.asarray(offs, dtype=np.uint64)
-        assert len(offs) % grid == 0
-        calls = len(offs) // grid
-        d_off = offs if isinstance(offs, torch.Tensor) else self._dev(offs.view(np.int64))
+        if isinstance(offs, torch.Tensor):
+            d_off = offs
+        else:
+            d_off = self._dev(np.asarray(offs, dtype=np.uint64).view(np.int64))
+        assert d_off.numel() % grid == 0
+        calls = d_off.numel() // grid
         if out is None:
             out = torch.zeros(2, dtype=torch.int64, device=dev)
         s, sp = self._stream(stream)

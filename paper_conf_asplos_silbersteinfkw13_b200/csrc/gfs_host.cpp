@@ -654,8 +654,11 @@ GFS_API int gfs_host_stats(gfs_handle* h, uint64_t* out, int n) {
 
 GFS_API int gfs_info(gfs_handle* h, uint64_t* out, int n) {
   if (!h || !out) return -EINVAL;
-  uint64_t v[7] = {h->h.page_size, h->h.nframes, h->h.max_files, h->h.max_nodes, h->h.ring_slots,
-                   h->workers.size(), h->wv64 ? 1u : 0u};
-  for (int i = 0; i < n && i < 7; ++i) out[i] = v[i];
-  return 7;
+  unsigned long long tail = 0;
+  cudaMemcpyAsync(&tail, h->h.ring_tail, 8, cudaMemcpyDeviceToHost, h->priv);
+  cudaStreamSynchronize(h->priv);
+  uint64_t v[9] = {h->h.page_size, h->h.nframes, h->h.max_files, h->h.max_nodes, h->h.ring_slots,
+                   h->workers.size(), h->wv64 ? 1u : 0u, h->next_ticket.load(), tail};
+  for (int i = 0; i < n && i < 9; ++i) out[i] = v[i];
+  return 9;
 }
