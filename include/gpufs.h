@@ -132,7 +132,9 @@ int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncall
                    uint32_t grid, uint32_t block);
 
 /* One-block file operations: op 0 = gfsync, 1 = gftruncate(arg), 2 = gfstat_size,
- * 3 = gopen+gclose only. flags = open flags. *d_ret = result. */
+ * 3 = gopen+gclose only, 4 = pin (gopen without gclose: the file stays open
+ * across launches, *d_ret = fd), 5 = unpin (gclose(fd = arg)).
+ * flags = open flags. *d_ret = result. */
 int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int flags, int op, uint64_t arg,
                    int64_t* d_ret);
 

@@ -130,8 +130,24 @@ __device__ __forceinline__ void backoff(uint32_t& ns) {
   ns = ns < 4096 ? ns * 2 : 4096;
 }
 
+// Relaxed, fence-free variants for the cache-hit fast path. On sm_100a an
+// acquire load/atomic compiles to LDG.STRONG + CCTL.IVALL (invalidates the
+// whole L1 of the SM) and a release to MEMBAR.ALL.GPU; the fast path instead
+// orders by address dependency and does all metadata accesses at L2.
+__device__ __forceinline__ uint32_t atom_add_rlx(uint32_t* p, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.relaxed.gpu.global.add.u32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ void red_add_rlx(uint32_t* p, uint32_t v) {
+  asm volatile("red.relaxed.gpu.global.add.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+__device__ __forceinline__ void red_add64(unsigned long long* p, unsigned long long v) {
+  asm volatile("red.relaxed.gpu.global.add.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+
 __device__ __forceinline__ void ctr(const gfs_ctx* c, int i, unsigned long long v = 1) {
-  atomicAdd(&c->ctr[(size_t)i * GFS_CTR_SHARDS + (smid() & (GFS_CTR_SHARDS - 1))], v);
+  red_add64(&c->ctr[(size_t)i * GFS_CTR_SHARDS + (smid() & (GFS_CTR_SHARDS - 1))], v);
 }
 
 __device__ __forceinline__ uint32_t stamp_now() { return (uint32_t)(now_ns() >> 10); }
@@ -157,6 +173,13 @@ struct Scratch {
   int64_t aux;
   void* ptr;
   FileSnap fs;
+  // Snapshot of the fd this block opened last: valid while the block holds it
+  // open (an open file cannot be re-incarnated). Shared memory is not cleared
+  // between launches or blocks, so the key includes %gridid and the block id.
+  FileSnap cached;
+  uint64_t cached_grid;
+  uint32_t cached_blk;
+  int32_t cached_fd;
   int32_t frame[GFS_MAX_BATCH];
   uint32_t installed[GFS_MAX_BATCH];
   int32_t err;
@@ -446,9 +469,18 @@ __device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx) {
   }
 }
 
+// Release after reading a frame: the block barrier before it guarantees every
+// load of the frame has returned (its consumer store could not issue
+// otherwise), so a relaxed decrement suffices.
 __device__ __forceinline__ void frame_release(const gfs_ctx* c, uint32_t f) {
   st_rlx(&c->f_stamp[f], stamp_now());
-  atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);  // ref - 1
+  red_add_rlx(&c->f_state[f], 0xFFFFFFFFu);  // ref - 1
+}
+// Release after writing a frame (gwrite): the dirty-range updates must be
+// visible before the reference drops (gfsync only syncs unreferenced frames).
+__device__ __forceinline__ void frame_release_rel(const gfs_ctx* c, uint32_t f) {
+  st_rlx(&c->f_stamp[f], stamp_now());
+  atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
 }
 
 // Give back a frame we installed but could not publish (lost the CAS race).
@@ -459,6 +491,36 @@ __device__ __forceinline__ void frame_abandon(const gfs_ctx* c, uint32_t f) {
 }
 
 // ------------------------------------------------------------------ page lookup
+// Cache-hit fast path (one optimistic attempt): relaxed walk
+// without creating nodes, relaxed incref, then the tag load made
+// address-dependent on the incref's result so it cannot be performed before
+// it (a plain relaxed load could be satisfied first and validate against a
+// tag the evictor has since replaced). All accesses are strong gpu-scope
+// operations served at L2, so no L1 line can be stale. Returns the frame, or
+// -1 to take the full (acquire/release) path.
+__device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
+  uint32_t node = fs.root;
+  for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
+    node = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
+    if (!node) return -1;
+  }
+  const uint32_t s = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
+  if (!s) return -1;
+  const uint32_t f = s - 1;
+  const uint32_t old = atom_add_rlx(&c->f_state[f], 1u);
+  // bit 30 of the state word is never set, so fdep == f; the dependency is real
+  const uint32_t fdep = min(f, f + (old & 0x40000000u));
+  const uint64_t tag = ld_rlx64(&c->f_tag[fdep]);
+  if (tag == (((uint64_t)fs.uid << 32) | (uint32_t)page) &&
+      !(old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
+    ctr(c, GFS_C_HIT);
+    ctr(c, GFS_C_LOCKFREE);
+    return (int)f;
+  }
+  red_add_rlx(&c->f_state[f], 0xFFFFFFFFu);
+  return -1;
+}
+
 // Find page `page` of the snapshot file and take a reference (P:L575-576,
 // P:L616-619). Lock-free: read slot, incref, validate tag == (uid,page)
 // (P:L669-672). Retries once without locking, then takes the file lock on
@@ -673,6 +735,25 @@ __device__ __forceinline__ bool snap_fd(const gfs_ctx* c, int fd, FileSnap* s) {
   return true;
 }
 
+__device__ __forceinline__ uint64_t grid_id() {
+  uint64_t g;
+  asm volatile("mov.u64 %0, %%gridid;" : "=l"(g));
+  return g;
+}
+__device__ __forceinline__ uint32_t block_linear() {
+  return blockIdx.x + gridDim.x * (blockIdx.y + gridDim.y * blockIdx.z);
+}
+
+// Snapshot for gread: read-only files this block opened are served from the
+// block's cached snapshot (their entry cannot change while held open).
+__device__ __forceinline__ bool snap_fd_cached(const gfs_ctx* c, Scratch& sc, int fd, FileSnap* s) {
+  if (sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id()) {
+    *s = sc.cached;
+    return true;
+  }
+  return snap_fd(c, fd, s);
+}
+
 // Write back every dirty, unreferenced page of the snapshot file in pages
 // [pb, pe), strided over the calling threads. Returns 0, -EBUSY (a dirty page
 // was mapped or in use, Tab.1), or a negative RPC error.
@@ -763,6 +844,12 @@ __device__ int new_incarnation(const gfs_ctx* c, gfs_file* e, uint32_t flags, co
   return 0;
 }
 
+// Move a file entry from state `from` to `to` (and adjust its count by dref)
+// with one atomic delta, preserving transient increments of other openers.
+__device__ __forceinline__ void sr_shift(gfs_file* e, uint32_t from, uint32_t to, int dref) {
+  atom_add_rel(&e->sr, (uint32_t)(((to - from) << 24) + (uint32_t)dref));
+}
+
 // gopen body, run by one thread.
 __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
   if (flags != (int)GFS_O_RDONLY && flags != (int)GFS_O_GWRONCE) return -EINVAL;
@@ -790,16 +877,18 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
       e->path_hash = h;
       e->lock = 0;
       e->err = 0;
-      st_rel(&e->sr, (GFS_FS_OPENING << 24) | 1u);
+      // From here on other openers may hold transient +1s on `sr` (fast path
+      // below): every state change is an atomic delta, never a plain store.
+      sr_shift(e, GFS_FS_CLAIM, GFS_FS_OPENING, 0);
       gfs_rpc_resp rs;
       int r = open_rpc_fill(c, e, i, (uint32_t)flags, 0, &rs);
       if (r == 0) r = new_incarnation(c, e, (uint32_t)flags, rs);
       if (r < 0) {
         e->err = r;
-        st_rel(&e->sr, GFS_FS_DEAD << 24);  // tombstone; a later gopen retries further along
+        sr_shift(e, GFS_FS_OPENING, GFS_FS_DEAD, -1);  // tombstone; a later gopen retries further along
         return r;
       }
-      st_rel(&e->sr, (GFS_FS_OPEN << 24) | 1u);
+      sr_shift(e, GFS_FS_OPENING, GFS_FS_OPEN, 0);
       return (int)i;
     }
     if (st == GFS_FS_CLAIM) {  // being inserted: wait for its path
@@ -823,15 +912,22 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
       continue;
     }
     if (st == GFS_FS_OPEN) {
-      if (e->oflags != (uint32_t)flags) return -EBUSY;  // one writer at a time
-      if (atom_cas(&e->sr, sr, sr + 1) == sr) {
-        ctr(c, GFS_C_OPEN_FAST);  // no CPU communication (P:L372-374)
+      if (ld_rlx(&e->oflags) != (uint32_t)flags) return -EBUSY;  // one writer at a time
+      // Fast path: a plain increment, no CAS loop — hundreds of
+      // blocks open the same file at once. Undo if the state moved meanwhile.
+      const uint32_t old = atom_add_acq(&e->sr, 1u);
+      if ((old >> 24) == GFS_FS_OPEN) {
+        ctr(c, GFS_C_OPEN_FAST);  // no CPU communication
         return (int)i;
       }
+      atom_add_rel(&e->sr, 0xFFFFFFFFu);
       continue;
     }
     if (st == GFS_FS_CLOSED) {
-      if (atom_cas(&e->sr, sr, (GFS_FS_REOPENING << 24) | 1u) != sr) continue;
+      if ((sr & 0xFFFFFF) != 0 || atom_cas(&e->sr, sr, (GFS_FS_REOPENING << 24) | 1u) != sr) {
+        backoff(ns);
+        continue;
+      }
       // Closed-file cache: re-open validates against the host (lazy
       // invalidation). O_GWRONCE or a mode change always starts
       // a fresh incarnation (pristine copy = zeros).
@@ -842,14 +938,14 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
         const uint64_t np = (old.size + c->page_size - 1) >> c->page_shift;
         int r = sync_pages(c, old, 0, np, 0, 1);
         if (r < 0 && r != -EBUSY) {
-          st_rel(&e->sr, GFS_FS_CLOSED << 24);
+          sr_shift(e, GFS_FS_REOPENING, GFS_FS_CLOSED, -1);
           return r;
         }
       }
       gfs_rpc_resp rs;
       int r = open_rpc_fill(c, e, i, (uint32_t)flags, old.hfid + 1u, &rs);
       if (r < 0) {
-        st_rel(&e->sr, GFS_FS_CLOSED << 24);
+        sr_shift(e, GFS_FS_REOPENING, GFS_FS_CLOSED, -1);
         return r;
       }
       const bool same = (uint32_t)flags == GFS_O_RDONLY && old.oflags == GFS_O_RDONLY &&
@@ -864,11 +960,11 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
         ctr(c, GFS_C_INVALIDATE);
         if (r < 0) {
           e->err = r;
-          st_rel(&e->sr, GFS_FS_DEAD << 24);
+          sr_shift(e, GFS_FS_REOPENING, GFS_FS_DEAD, -1);
           return r;
         }
       }
-      st_rel(&e->sr, (GFS_FS_OPEN << 24) | 1u);
+      sr_shift(e, GFS_FS_REOPENING, GFS_FS_OPEN, 0);
       return (int)i;
     }
     i = (i + 1) & mask;  // unknown state: skip
@@ -876,15 +972,18 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
   }
 }
 
+// gclose body: decrement; the holder that drops the count to zero moves the
+// entry to the closed-file table unless it was re-opened meanwhile.
 __device__ int close_leader(const gfs_ctx* c, int fd) {
   if (fd < 0 || (uint32_t)fd >= c->max_files) return -EBADF;
   gfs_file* e = c->files + fd;
-  for (;;) {
-    const uint32_t sr = ld_acq(&e->sr);
-    if ((sr >> 24) != GFS_FS_OPEN || (sr & 0xFFFFFF) == 0) return -EBADF;
-    const uint32_t nsr = (sr & 0xFFFFFF) == 1 ? (GFS_FS_CLOSED << 24) : sr - 1;
-    if (atom_cas(&e->sr, sr, nsr) == sr) return 0;  // no write-back
+  const uint32_t old = atom_add_rel(&e->sr, 0xFFFFFFFFu);
+  if ((old >> 24) != GFS_FS_OPEN || (old & 0xFFFFFF) == 0) {
+    atom_add_rel(&e->sr, 1u);
+    return -EBADF;
   }
+  if ((old & 0xFFFFFF) == 1) atom_cas(&e->sr, GFS_FS_OPEN << 24, GFS_FS_CLOSED << 24);
+  return 0;  // no write-back
 }
 
 }  // namespace detail
@@ -896,7 +995,16 @@ using detail::Scratch;
 __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
   Scratch& sc = detail::scratch();
   __syncthreads();
-  if (detail::block_tid() == 0) sc.ret = detail::open_leader(c, path, flags);
+  if (detail::block_tid() == 0) {
+    const int fd = detail::open_leader(c, path, flags);
+    sc.ret = fd;
+    sc.cached_fd = -1;
+    if (fd >= 0 && detail::snap_fd(c, fd, &sc.cached) && !(sc.cached.oflags & GFS_O_GWRONCE)) {
+      sc.cached_grid = detail::grid_id();
+      sc.cached_blk = detail::block_linear();
+      sc.cached_fd = fd;
+    }
+  }
   __syncthreads();
   return (int)sc.ret;
 }
@@ -905,7 +1013,10 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
 __device__ inline int gclose(const gfs_ctx* c, int fd) {
   Scratch& sc = detail::scratch();
   __syncthreads();
-  if (detail::block_tid() == 0) sc.ret = detail::close_leader(c, fd);
+  if (detail::block_tid() == 0) {
+    if (sc.cached_fd == fd) sc.cached_fd = -1;
+    sc.ret = detail::close_leader(c, fd);
+  }
   __syncthreads();
   return (int)sc.ret;
 }
@@ -926,33 +1037,58 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   using namespace detail;
   Scratch& sc = scratch();
   const int tid = block_tid(), nthr = block_nthr();
-  __syncthreads();
-  if (tid == 0) {
-    FileSnap s;
-    if (!snap_fd(c, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
-      sc.ret = -EBADF;
-    } else {
-      sc.fs = s;
-      sc.ret = off >= s.size ? 0 : (int64_t)(len < s.size - off ? len : s.size - off);
-      ctr(c, GFS_C_GREAD_CALLS);
-      if (sc.ret > 0) ctr(c, GFS_C_GREAD_BYTES, (unsigned long long)sc.ret);
+  const uint32_t shift = c->page_shift;
+  const uint64_t P = c->page_size;
+  const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
+  __syncthreads();  // the call is a barrier: earlier uses of dst by the block are complete
+  // Warp 0 alone: snapshot + clip, then the first batch of lookups (one page
+  // per lane). Other warps only touch `sc` after the next barrier.
+  if (tid < 32) {
+    if (tid == 0) {
+      FileSnap s;
+      if (!snap_fd_cached(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
+        sc.ret = -EBADF;
+      } else {
+        sc.fs = s;
+        sc.ret = off >= s.size ? 0 : (int64_t)(len < s.size - off ? len : s.size - off);
+        ctr(c, GFS_C_GREAD_CALLS);
+        if (sc.ret > 0) ctr(c, GFS_C_GREAD_BYTES, (unsigned long long)sc.ret);
+      }
+    }
+    __syncwarp(nthr >= 32 ? 0xFFFFFFFFu : ((1u << nthr) - 1u));
+    const int64_t n0 = sc.ret;
+    if (n0 > 0) {
+      const uint64_t q0 = off >> shift, q1 = (off + (uint64_t)n0 - 1) >> shift;
+      const uint32_t cnt = (uint32_t)((q1 - q0 + 1) < B ? (q1 - q0 + 1) : B);
+      if (tid < (int)cnt) {
+        const FileSnap fs0 = sc.fs;
+        int f = (c->flags & GFS_F_LOCKED_TRAVERSAL) ? -1 : lookup_fast(c, fs0, q0 + tid);
+        if (f < 0) {
+          uint32_t inst;
+          f = lookup_page(c, fs0, q0 + tid, &inst);
+        }
+        sc.frame[tid] = f;
+      }
     }
   }
   __syncthreads();
   const int64_t n = sc.ret;
   if (n <= 0) return n;
   const FileSnap fs = sc.fs;
-  const uint32_t shift = c->page_shift;
-  const uint64_t P = c->page_size;
   const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
-  const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
   for (uint64_t pb = p0; pb <= p1; pb += B) {
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
-    if (tid < (int)cnt) {
-      uint32_t inst;
-      sc.frame[tid] = lookup_page(c, fs, pb + tid, &inst);
+    if (pb != p0) {  // later batches: lookups by the first cnt threads
+      if (tid < (int)cnt) {
+        int f = (c->flags & GFS_F_LOCKED_TRAVERSAL) ? -1 : lookup_fast(c, fs, pb + tid);
+        if (f < 0) {
+          uint32_t inst;
+          f = lookup_page(c, fs, pb + tid, &inst);
+        }
+        sc.frame[tid] = f;
+      }
+      __syncthreads();
     }
-    __syncthreads();
     int err = 0;
     for (uint32_t i = 0; i < cnt; ++i)
       if (sc.frame[i] < 0) err = sc.frame[i];
@@ -961,8 +1097,9 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
         const uint64_t p = pb + i;
         const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
         const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-        block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
-                              e - s, tid, nthr);
+        uint8_t* d = (uint8_t*)dst + ((p << shift) + s - off);
+        const uint8_t* src = frame_ptr(c, (uint32_t)sc.frame[i]) + s;
+        block_copy_from_frame(d, src, e - s, tid, nthr);
       }
     }
     __syncthreads();
@@ -1038,7 +1175,7 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
         atomicAdd(&c->f_written[f], e - s);
       }
       if (sc.installed[tid]) atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
-      frame_release(c, f);
+      frame_release_rel(c, f);
     }
     if (err) return err;
   }

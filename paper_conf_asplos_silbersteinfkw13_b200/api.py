@@ -164,12 +164,19 @@ class GpuFS:
     def fileop(self, path, op, flags=0, arg=0, stream=None) -> int:
         """op: 'fsync' | 'ftruncate' | 'fstat' | 'openclose'."""
         torch = _torch()
-        code = {"fsync": 0, "ftruncate": 1, "fstat": 2, "openclose": 3}[op]
+        code = {"fsync": 0, "ftruncate": 1, "fstat": 2, "openclose": 3, "pin": 4, "unpin": 5}[op]
         d_ret = torch.full((1,), -999, dtype=torch.int64, device=f"cuda:{self.device}")
         s, sp = self._stream(stream)
         gfs_run_fileop(self.h, sp, path, flags, code, arg, d_ret.data_ptr())
         s.synchronize()
         return int(d_ret.item())
+
+    def pin(self, path, flags=0) -> int:
+        """Open `path` and keep it open across launches (later gopen calls need no RPC)."""
+        return self.fileop(path, "pin", flags=flags)
+
+    def unpin(self, fd) -> int:
+        return self.fileop("", "unpin", arg=fd)
 
     def gfsync(self, path):
         return self.fileop(path, "fsync", flags=1)

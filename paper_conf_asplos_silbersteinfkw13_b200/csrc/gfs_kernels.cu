@@ -124,7 +124,7 @@ __global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint
   if (fd >= 0) gclose(c, fd);
 }
 
-__global__ void k_seqread(const gfs_ctx* c, const char* path, uint64_t file_off, uint64_t total, uint64_t chunk,
+__global__ void __launch_bounds__(256, 4) k_seqread(const gfs_ctx* c, const char* path, uint64_t file_off, uint64_t total, uint64_t chunk,
                           int use_mmap, uint8_t* scratch, uint64_t* sum, int64_t* err) {
   const int tid = threadIdx.x, nthr = blockDim.x;
   const int fd = gopen(c, path, GFS_O_RDONLY);
@@ -168,7 +168,7 @@ __global__ void k_seqread(const gfs_ctx* c, const char* path, uint64_t file_off,
   gclose(c, fd);
 }
 
-__global__ void k_randread(const gfs_ctx* c, const char* path, int raw, const uint8_t* rawp, uint32_t chunk,
+__global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const char* path, int raw, const uint8_t* rawp, uint32_t chunk,
                            uint32_t calls, const uint64_t* offs, uint64_t* sum, int64_t* err) {
   extern __shared__ __align__(16) uint8_t smem[];
   const int tid = threadIdx.x, nthr = blockDim.x;
@@ -215,6 +215,11 @@ __global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncal
 }
 
 __global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, uint64_t arg, int64_t* ret) {
+  if (op == 5) {  // unpin: drop a reference taken by op 4
+    const int64_t r = gclose(c, (int)arg);
+    if (threadIdx.x == 0) *ret = r;
+    return;
+  }
   const int fd = gopen(c, path, flags);
   int64_t r = fd;
   if (fd >= 0) {
@@ -222,8 +227,10 @@ __global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, 
     else if (op == 1) r = gftruncate(c, fd, arg);
     else if (op == 2) r = gfstat_size(c, fd);
     else r = fd;
-    const int cr = gclose(c, fd);
-    if (r >= 0 && cr < 0) r = cr;
+    if (op != 4) {  // op 4 = pin: keep the file open across launches
+      const int cr = gclose(c, fd);
+      if (r >= 0 && cr < 0) r = cr;
+    }
   }
   if (threadIdx.x == 0) *ret = r;
 }
