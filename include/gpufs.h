@@ -43,7 +43,7 @@ typedef struct gfs_config {
   uint32_t max_nodes;       /* radix node pool (0 = auto) */
   uint32_t max_batch;       /* pages looked up per warp-0 batch, 1..32 */
   uint32_t flags;           /* GFS_F_* (gpufs_layout.h) */
-  uint32_t pad;
+  uint32_t staging_slots;   /* pinned host staging slots of page_size bytes (0 = auto: 128 MiB worth) */
   uint64_t timeout_ms;      /* device-side wait bound (0 = none) -> -ETIMEDOUT */
   void* frame_pool;         /* optional caller-owned device memory >= cache_bytes */
 } gfs_config;
@@ -137,6 +137,42 @@ int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncall
  * flags = open flags. *d_ret = result. */
 int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int flags, int op, uint64_t arg,
                    int64_t* d_ret);
+
+/* --------------------------------------------------------------------------
+ * grep -w consumer (§5.2.2): for each word of the dictionary
+ * (one word per 32-byte slot) count how many times and in which
+ * files it appears; the input file names are read from the
+ * list file (one path per line, relative to the list's directory,
+ * P:L1266-1267). Word bytes are [A-Za-z0-9_]; counts are per occurrence.
+ * ------------------------------------------------------------------------ */
+typedef struct gfs_grep_params {
+  uint32_t max_files;   /* capacity of the file list */
+  uint32_t max_words;   /* capacity of the dictionary (words) */
+  uint64_t list_cap;    /* bytes of the list file (capacity) */
+  uint64_t pair_cap;    /* (file, word) table slots (rounded up to a power of two) */
+  uint64_t hit_cap;     /* hits to list in d_hits (0: none) */
+  uint32_t chunk;       /* work-item bytes, multiple of 16 */
+  uint32_t grid;        /* persistent blocks */
+  uint32_t block;       /* threads per block, multiple of 32, <= 256 */
+  uint32_t keep_open;   /* 1: leave every file open after the run (warm re-runs skip the host) */
+} gfs_grep_params;
+
+/* Device scratch bytes gfs_grep needs for these parameters. */
+uint64_t gfs_grep_work_bytes(const gfs_grep_params* p);
+
+/* Enqueue the whole search on `stream`. Outputs (device memory, caller-owned):
+ *   d_rec[3*i .. 3*i+2] = (file index, word index, count), unique pairs, unordered,
+ *                         up to rec_cap records (d_summary[0] = records found);
+ *   d_totals[k]         = occurrences of word k over all files (max_words entries);
+ *   d_hits[2*i], [2*i+1] = ((file << 32) | word, byte offset) per hit if non-NULL,
+ *                         up to hit_cap (d_summary[8] = hits listed + dropped);
+ *   d_summary[0..9]     = nrecords, nhits, digest_sum, digest_xor, nfiles, nwords,
+ *                         corpus bytes, error (0 or -errno), nhits_listed, nitems.
+ * The digest is sum and xor over hits of splitmix64(splitmix64(splitmix64(f)+off)+k)
+ * (order independent). File index = position among the list's non-empty lines. */
+int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
+             const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
+             uint64_t* d_hits, uint64_t* d_summary);
 
 #ifdef __cplusplus
 }

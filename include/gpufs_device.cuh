@@ -18,7 +18,9 @@
 // the same function with the same arguments at the same point; each call is an
 // implicit barrier and every thread receives the same return value. Negative
 // returns are -errno. `dst`/`src` may point to global or shared memory and are
-// owned by the caller. A gmmap pointer is borrowed until gmunmap.
+// owned by the caller. A gmmap pointer is borrowed until gmunmap. fds are
+// GPU-global (an fd names a file): a block may use an fd another
+// block opened while that open is held.
 //
 // Errors: -EBADF bad/closed fd, gread on O_GWRONCE, gwrite on O_RDONLY;
 // -EINVAL bad flags; -ENOENT/-EACCES from host open; -EMFILE table full;
@@ -29,21 +31,29 @@
 //
 // Design: per-file radix tree (fanout 256) of u32 frame ids in
 // HBM, looked up lock-free with (uid,page) tag validation; frame
-// state word with refcount + FILLING/EVICTING bits; misses install a frame by
-// CAS, post an RPC on the pinned ring and wait on a device-memory completion
-// word written by the host daemon's stream after its DMA;
-// eviction is a sampled, tiered LRU over 32-frame windows run in the calling
-// thread. Slots are hints: evictors never touch tree nodes, a
-// reader that finds a stale slot installs over it.
+// state word = refcount + FILLING/EVICTING/ERROR bits, changed only by atomic
+// deltas. A miss installs a frame by CAS and posts an RPC on the pinned ring
+// (P:L719-725); the host daemon preads into a pinned staging slot and stores a
+// completion word in pinned memory; the installing BLOCK then pulls the page
+// over PCIe into the frame and clears FILLING. No CUDA stream operation is on
+// the miss path (a stream-ordered DMA can sit behind the running kernel in a
+// shared hardware queue). Lookups never wait on another block's fill: they
+// report BUSY and the block retries after filling its own pages, so blocks
+// never wait on each other in a cycle. Eviction is a sampled, tiered LRU over
+// 32-frame windows run in the calling thread. Tree slots are
+// hints: evictors never touch tree nodes; a reader that finds a stale slot
+// installs over it.
 #pragma once
 
 #include <stdint.h>
 #include <errno.h>
 #include "gpufs_layout.h"
 
-
 namespace gfs {
 namespace detail {
+namespace {  // internal linkage: the header is included by several translation units
+
+constexpr int kBusy = -10000;  // lookup result: page being filled/evicted elsewhere
 
 // ------------------------------------------------------------------ PTX
 __device__ __forceinline__ uint64_t now_ns() {
@@ -122,14 +132,6 @@ __device__ __forceinline__ uint32_t atom_cas(uint32_t* p, uint32_t cmp, uint32_t
                : "=r"(r) : "l"(p), "r"(cmp), "r"(val) : "memory");
   return r;
 }
-__device__ __forceinline__ unsigned long long atom_add64(unsigned long long* p, unsigned long long v) {
-  return atomicAdd(p, v);
-}
-__device__ __forceinline__ void backoff(uint32_t& ns) {
-  __nanosleep(ns);
-  ns = ns < 4096 ? ns * 2 : 4096;
-}
-
 // Relaxed, fence-free variants for the cache-hit fast path. On sm_100a an
 // acquire load/atomic compiles to LDG.STRONG + CCTL.IVALL (invalidates the
 // whole L1 of the SM) and a release to MEMBAR.ALL.GPU; the fast path instead
@@ -144,6 +146,15 @@ __device__ __forceinline__ void red_add_rlx(uint32_t* p, uint32_t v) {
 }
 __device__ __forceinline__ void red_add64(unsigned long long* p, unsigned long long v) {
   asm volatile("red.relaxed.gpu.global.add.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ unsigned long long atom_add64(unsigned long long* p, unsigned long long v) {
+  unsigned long long r;
+  asm volatile("atom.relaxed.gpu.global.add.u64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ void backoff(uint32_t& ns) {
+  __nanosleep(ns);
+  ns = ns < 4096 ? ns * 2 : 4096;
 }
 
 __device__ __forceinline__ void ctr(const gfs_ctx* c, int i, unsigned long long v = 1) {
@@ -161,6 +172,14 @@ __device__ __forceinline__ int block_tid() {
   return threadIdx.x + blockDim.x * (threadIdx.y + blockDim.y * threadIdx.z);
 }
 __device__ __forceinline__ int block_nthr() { return blockDim.x * blockDim.y * blockDim.z; }
+__device__ __forceinline__ uint64_t grid_id() {
+  uint64_t g;
+  asm volatile("mov.u64 %0, %%gridid;" : "=l"(g));
+  return g;
+}
+__device__ __forceinline__ uint32_t block_linear() {
+  return blockIdx.x + gridDim.x * (blockIdx.y + gridDim.y * blockIdx.z);
+}
 
 // ------------------------------------------------------------------ scratch
 struct FileSnap {
@@ -180,8 +199,11 @@ struct Scratch {
   uint64_t cached_grid;
   uint32_t cached_blk;
   int32_t cached_fd;
-  int32_t frame[GFS_MAX_BATCH];
-  uint32_t installed[GFS_MAX_BATCH];
+  int32_t frame[GFS_MAX_BATCH];   // >= 0 held frame; kBusy / -errno otherwise
+  int32_t stage[GFS_MAX_BATCH];   // staging slot to pull from (>= 0), or -1
+  uint32_t fill[GFS_MAX_BATCH];   // 1: this block installed the frame and must fill it
+  uint32_t nbytes[GFS_MAX_BATCH]; // valid bytes of a filled page
+  uint32_t lo[GFS_MAX_BATCH], hi[GFS_MAX_BATCH];
   int32_t err;
   uint32_t busy;
 };
@@ -191,14 +213,51 @@ __device__ __forceinline__ Scratch& scratch() {
   return s;
 }
 
+// ------------------------------------------------------------------ staging slots
+// Pinned host memory, page_size bytes per slot, device-mapped; a bitmap in HBM
+// hands slots out. A slot is held only across one RPC and the copy around it,
+// never while waiting on another block, so allocation always makes progress.
+__device__ int stage_alloc(const gfs_ctx* c) {
+  const uint32_t W = c->staging_words;
+  uint32_t w = (smid() * 7u + (uint32_t)(now_ns() >> 6)) % W;
+  const uint64_t t0 = now_ns();
+  uint32_t ns = 64;
+  bool waited = false;
+  for (uint32_t pass = 0;; ++pass) {
+    for (uint32_t k = 0; k < W; ++k, w = (w + 1 == W ? 0 : w + 1)) {
+      uint32_t cur = ld_rlx(c->staging_bits + w);
+      while (cur != 0xFFFFFFFFu) {
+        const uint32_t bit = __ffs(~cur) - 1;
+        const uint32_t idx = w * 32 + bit;
+        if (idx >= c->staging_slots) break;
+        const uint32_t prev = atomicOr(c->staging_bits + w, 1u << bit);
+        if (!(prev & (1u << bit))) {
+          if (waited) ctr(c, GFS_C_STAGE_WAIT);
+          return (int)idx;
+        }
+        cur = prev | (1u << bit);
+      }
+    }
+    waited = true;
+    backoff(ns);
+    if (timed_out(c, t0)) return -ETIMEDOUT;
+  }
+}
+__device__ __forceinline__ void stage_free(const gfs_ctx* c, int idx) {
+  atomicAnd(c->staging_bits + (idx >> 5), ~(1u << (idx & 31)));
+}
+__device__ __forceinline__ uint8_t* stage_ptr(const gfs_ctx* c, int idx) {
+  return c->staging + ((size_t)idx << c->page_shift);
+}
+
 // ------------------------------------------------------------------ RPC client
 // One request on the per-GPU queue: take a ticket, fill the 64-byte
 // slot in pinned host memory, publish seq with st.release.sys (the GPU->CPU
-// fence), then wait for the completion word in HBM that the
-// daemon's stream writes after its DMA. Any thread may call.
-__device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64_t file_off,
-                            uint64_t dev_ptr, uint32_t len, uint32_t flags, uint64_t arg,
-                            const char* path, uint32_t path_len, gfs_rpc_resp* resp_out) {
+// fence), then poll the completion word the host stores in pinned
+// memory (ld.acquire.sys: P:L693-696's cache bypass). Any thread may call.
+__device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64_t file_off, int stage,
+                            uint32_t len, uint32_t flags, uint64_t arg, const char* path, uint32_t path_len,
+                            gfs_rpc_resp* resp_out) {
   const unsigned long long t = atom_add64(c->ring_tail, 1ull);
   const uint32_t R = c->ring_slots;
   const uint32_t slot = (uint32_t)(t % R);
@@ -221,11 +280,12 @@ __device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64
   q->op = op;
   q->hfid = hfid;
   q->file_off = file_off;
-  q->dev_ptr = dev_ptr;
+  q->dev_ptr = 0;
   q->len = len;
   q->flags = flags;
   q->arg = arg;
   q->path_len = path_len;
+  q->stage = (uint32_t)stage;
   if (path) {
     volatile char* dp = c->ring_paths + (size_t)slot * GFS_MAX_PATH;
     for (uint32_t i = 0; i < path_len; ++i) dp[i] = path[i];
@@ -303,8 +363,7 @@ __device__ void tree_free(const gfs_ctx* c, uint32_t root, uint32_t height) {
   int sp = 0;
   stk_node[0] = root;
   stk_idx[0] = 0;
-  // levels: stack depth d corresponds to node height (height - d)
-  while (sp >= 0) {
+  while (sp >= 0) {  // stack depth d holds a node of height (height - d)
     const uint32_t node = stk_node[sp];
     const uint32_t h = height - (uint32_t)sp;
     if (h > 1 && stk_idx[sp] < GFS_FANOUT) {
@@ -360,6 +419,89 @@ __device__ __forceinline__ uint32_t height_for(uint64_t npages) {
   return 4;
 }
 
+// ------------------------------------------------------------------ copies
+// Block-cooperative copy of n bytes. Frame reads bypass L1 (ld.global.cg):
+// a frame may have been refilled since this SM last cached it.
+// 16-byte vectors with 4 loads in flight per thread when src/dst are
+// co-aligned; 4-byte or byte fallback otherwise.
+template <bool kHostSrc>
+__device__ __forceinline__ uint8_t ld_b(const uint8_t* p) {
+  return kHostSrc ? __ldcv(p) : __ldcg(p);
+}
+template <bool kHostSrc>
+__device__ __forceinline__ int4 ld_v(const int4* p) {
+  return kHostSrc ? __ldcv(p) : __ldcg(p);
+}
+template <bool kHostSrc>
+__device__ __forceinline__ uint32_t ld_w(const uint32_t* p) {
+  return kHostSrc ? __ldcv(p) : __ldcg(p);
+}
+
+template <bool kHostSrc = false>
+__device__ __forceinline__ void block_copy_from_frame(uint8_t* dst, const uint8_t* src, uint64_t n, int tid,
+                                                      int nthr) {
+  if (n == 0) return;
+  if ((((uintptr_t)src ^ (uintptr_t)dst) & 15) == 0) {
+    const uint64_t h0 = (16 - ((uintptr_t)src & 15)) & 15;
+    const uint64_t head = h0 < n ? h0 : n;
+    for (uint64_t i = tid; i < head; i += nthr) dst[i] = ld_b<kHostSrc>(src + i);
+    const uint64_t nv = (n - head) >> 4;
+    const int4* s4 = (const int4*)(src + head);
+    int4* d4 = (int4*)(dst + head);
+    uint64_t i = tid;
+    const uint64_t stride = (uint64_t)nthr;
+    for (; i + 3 * stride < nv; i += 4 * stride) {
+      int4 a = ld_v<kHostSrc>(s4 + i), b = ld_v<kHostSrc>(s4 + i + stride),
+           cc = ld_v<kHostSrc>(s4 + i + 2 * stride), d = ld_v<kHostSrc>(s4 + i + 3 * stride);
+      d4[i] = a;
+      d4[i + stride] = b;
+      d4[i + 2 * stride] = cc;
+      d4[i + 3 * stride] = d;
+    }
+    for (; i < nv; i += stride) d4[i] = ld_v<kHostSrc>(s4 + i);
+    const uint64_t done = head + (nv << 4);
+    for (uint64_t k = done + tid; k < n; k += nthr) dst[k] = ld_b<kHostSrc>(src + k);
+  } else if ((((uintptr_t)src ^ (uintptr_t)dst) & 3) == 0) {
+    const uint64_t h0 = (4 - ((uintptr_t)src & 3)) & 3;
+    const uint64_t head = h0 < n ? h0 : n;
+    for (uint64_t i = tid; i < head; i += nthr) dst[i] = ld_b<kHostSrc>(src + i);
+    const uint64_t nw = (n - head) >> 2;
+    const uint32_t* s4 = (const uint32_t*)(src + head);
+    uint32_t* d4 = (uint32_t*)(dst + head);
+    for (uint64_t i = tid; i < nw; i += nthr) d4[i] = ld_w<kHostSrc>(s4 + i);
+    for (uint64_t k = head + (nw << 2) + tid; k < n; k += nthr) dst[k] = ld_b<kHostSrc>(src + k);
+  } else {
+    for (uint64_t i = tid; i < n; i += nthr) dst[i] = ld_b<kHostSrc>(src + i);
+  }
+}
+
+// Copy into a frame or staging slot from user data / a frame (plain loads).
+__device__ __forceinline__ void block_copy_plain(uint8_t* dst, const uint8_t* src, uint64_t n, int tid, int nthr) {
+  if (n == 0) return;
+  if ((((uintptr_t)src ^ (uintptr_t)dst) & 15) == 0) {
+    const uint64_t h0 = (16 - ((uintptr_t)src & 15)) & 15;
+    const uint64_t head = h0 < n ? h0 : n;
+    for (uint64_t i = tid; i < head; i += nthr) dst[i] = src[i];
+    const uint64_t nv = (n - head) >> 4;
+    const int4* s4 = (const int4*)(src + head);
+    int4* d4 = (int4*)(dst + head);
+    for (uint64_t i = tid; i < nv; i += nthr) d4[i] = s4[i];
+    for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = src[k];
+  } else {
+    for (uint64_t i = tid; i < n; i += nthr) dst[i] = src[i];
+  }
+}
+
+__device__ __forceinline__ void block_zero(uint8_t* dst, uint64_t n, int tid, int nthr) {
+  const uint64_t h0 = (16 - ((uintptr_t)dst & 15)) & 15;
+  const uint64_t head = h0 < n ? h0 : n;
+  for (uint64_t i = tid; i < head; i += nthr) dst[i] = 0;
+  const uint64_t nv = (n - head) >> 4;
+  int4* d4 = (int4*)(dst + head);
+  for (uint64_t k = tid; k < nv; k += nthr) d4[k] = make_int4(0, 0, 0, 0);
+  for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = 0;
+}
+
 // ------------------------------------------------------------------ frames
 __device__ __forceinline__ uint8_t* frame_ptr(const gfs_ctx* c, uint32_t f) {
   return c->pool + ((size_t)f << c->page_shift);
@@ -379,21 +521,27 @@ __device__ __forceinline__ void frame_init(const gfs_ctx* c, uint32_t f, uint64_
   atom_add_rel(&c->f_state[f], GFS_ST_FILLING + 1u - GFS_ST_EVICTING);
 }
 
-// Write back a frame's dirty range (caller owns it: EVICTING, ref 0).
-__device__ int32_t frame_writeback(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
+// Write back a frame's dirty range from one thread (the caller owns the frame:
+// EVICTING, ref 0): copy it into a staging slot over PCIe, then WRITE RPC.
+__device__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
   const uint32_t lo = ld_rlx(&c->f_lo[f]);
   if (lo == GFS_DIRTY_NONE) return 0;
   const uint32_t hi = ld_rlx(&c->f_hi[f]);
   const uint32_t wr = ld_rlx(&c->f_written[f]);
   const uint64_t page = ld_rlx64(&c->f_tag[f]) & 0xFFFFFFFFull;
-  const uint64_t base = page << c->page_shift;
-  const int32_t r = rpc_call(c, GFS_OP_WRITE, hfid, base + lo, (uint64_t)(frame_ptr(c, f) + lo), hi - lo,
+  const int st = stage_alloc(c);
+  if (st < 0) return st;
+  block_copy_plain(stage_ptr(c, st) + lo, frame_ptr(c, f) + lo, hi - lo, 0, 1);
+  __threadfence_system();
+  const int32_t r = rpc_call(c, GFS_OP_WRITE, hfid, (page << c->page_shift) + lo, st, hi - lo,
                              wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, nullptr);
+  stage_free(c, st);
   if (r < 0) return r;
   st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
   st_rlx(&c->f_hi[f], 0);
   st_rlx(&c->f_written[f], 0);
   ctr(c, GFS_C_WRITEBACK);
+  ctr(c, GFS_C_RPC_WRITE);
   ctr(c, GFS_C_BYTES_D2H, hi - lo);
   return 0;
 }
@@ -449,7 +597,7 @@ __device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx) {
       const uint32_t f = (uint32_t)best;
       if (ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) {
         const uint32_t fi = ld_rlx(&c->f_file[f]);
-        const int32_t r = frame_writeback(c, f, ld_rlx(&c->files[fi].hfid));
+        const int32_t r = frame_writeback_lane(c, f, ld_rlx(&c->files[fi].hfid));
         if (r < 0) {  // keep the dirty page, try another victim
           atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
           continue;
@@ -521,15 +669,24 @@ __device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs,
   return -1;
 }
 
+struct Lk {
+  int frame;   // >= 0 held (ref taken); kBusy; or -errno
+  int stage;   // >= 0: pull nbytes from this staging slot into the frame
+  uint32_t fill;
+  uint32_t nbytes;
+};
+
 // Find page `page` of the snapshot file and take a reference (P:L575-576,
 // P:L616-619). Lock-free: read slot, incref, validate tag == (uid,page)
 // (P:L669-672). Retries once without locking, then takes the file lock on
-// the third attempt. A miss installs a frame by CAS and fills it:
-// READ RPC for O_RDONLY files, or (O_GWRONCE, never fetched) it
-// is returned with *installed = 1 and FILLING still set — the caller's block
-// zero-fills/writes it and clears FILLING.
-__device__ int lookup_page(const gfs_ctx* c, const FileSnap& fs, uint64_t page, uint32_t* installed) {
-  *installed = 0;
+// the third attempt. Never waits on another block: a page being
+// filled or evicted elsewhere returns kBusy. A miss installs a frame by CAS
+// and returns it with fill = 1 and FILLING still set: for O_RDONLY files the
+// page has been pread by the host into staging slot `stage` (READ RPC,
+// P:L570-576); for O_GWRONCE files nothing is fetched. The
+// caller's block fills the frame and clears FILLING.
+__device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
+  Lk out{kBusy, -1, 0, 0};
   const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)page;
   uint32_t* lockp = &c->files[fs.fdx].lock;
   bool locked = false;
@@ -541,58 +698,35 @@ __device__ int lookup_page(const gfs_ctx* c, const FileSnap& fs, uint64_t page, 
   uint32_t* slot = walk(c, fs.root, fs.height, page, true, &err);
   if (!slot) {
     if (locked) spin_unlock(lockp);
-    return err ? err : -ENOMEM;
+    out.frame = err ? err : -ENOMEM;
+    return out;
   }
-  const uint64_t t0 = now_ns();
   int attempt = 0;
-  int result;
   for (;;) {
     if (!locked && attempt >= 2) {
       spin_lock(lockp);
       locked = true;
     }
-    if (timed_out(c, t0)) {
-      ctr(c, GFS_C_TIMEOUT);
-      result = -ETIMEDOUT;
-      break;
-    }
     const uint32_t s = ld_acq(slot);
     if (s) {
       const uint32_t f = s - 1;
       const uint32_t old = atom_add_acq(&c->f_state[f], 1u);
-      uint64_t tag = ld_acq64(&c->f_tag[f]);
-      if (tag == want && !(old & GFS_ST_EVICTING)) {
-        uint32_t st = old;
-        uint32_t ns = 128;
-        while (st & GFS_ST_FILLING) {
-          backoff(ns);
-          st = ld_acq(&c->f_state[f]);
-          if (timed_out(c, t0)) break;
-        }
-        tag = ld_acq64(&c->f_tag[f]);
-        if (tag == want && !(st & (GFS_ST_ERROR | GFS_ST_FILLING))) {
+      const uint64_t tag = ld_acq64(&c->f_tag[f]);
+      if (tag == want) {
+        if (!(old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
           ctr(c, GFS_C_HIT);
-          result = (int)f;
+          out.frame = (int)f;
           break;
         }
         atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
-        if (tag == want && (st & GFS_ST_ERROR) && (old & GFS_ST_FILLING)) {
-          result = -EIO;  // the fill we waited for failed
+        if (old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
+          ctr(c, GFS_C_BUSY);
+          out.frame = kBusy;
           break;
         }
-        if (st & GFS_ST_FILLING) continue;  // timed out; loop reports it
+        // ERROR with no fill in flight: stale, install over it
       } else {
         atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
-        if (tag == want) {  // being synced or evicted: wait for it to settle
-          uint32_t ns = 128;
-          while (ld_acq64(&c->f_tag[f]) == want && (ld_acq(&c->f_state[f]) & GFS_ST_EVICTING)) {
-            backoff(ns);
-            if (timed_out(c, t0)) break;
-          }
-          ++attempt;
-          ctr(c, GFS_C_RETRY);
-          continue;
-        }
       }
       ++attempt;
       ctr(c, GFS_C_RETRY);
@@ -600,7 +734,7 @@ __device__ int lookup_page(const gfs_ctx* c, const FileSnap& fs, uint64_t page, 
     // miss (or stale slot): install a new frame for `want`
     const int g = alloc_frame(c, want, fs.fdx);
     if (g < 0) {
-      result = g;
+      out.frame = g;
       break;
     }
     if (atom_cas(slot, s, (uint32_t)g + 1u) != s) {
@@ -609,106 +743,129 @@ __device__ int lookup_page(const gfs_ctx* c, const FileSnap& fs, uint64_t page, 
       ctr(c, GFS_C_RETRY);
       continue;
     }
+    out.frame = g;
+    out.fill = 1;
     if (fs.oflags & GFS_O_GWRONCE) {
-      *installed = 1;
       ctr(c, GFS_C_ZERO_FILL);
-      result = g;
       break;
     }
-    // Fetch min(P, S - pP) bytes from the host into the frame.
+    // Fetch min(P, S - pP) bytes: the host preads into a staging slot.
     const uint64_t base = page << c->page_shift;
     const uint64_t rem = fs.size > base ? fs.size - base : 0;
     const uint32_t nb = (uint32_t)(rem < c->page_size ? rem : c->page_size);
-    const int32_t r = rpc_call(c, GFS_OP_READ, fs.hfid, base, (uint64_t)frame_ptr(c, (uint32_t)g), nb, 0, 0,
-                               nullptr, 0, nullptr);
+    const int st = nb ? stage_alloc(c) : -1;
+    int32_t r = st < 0 && nb ? st : 0;
+    if (nb && st >= 0) r = rpc_call(c, GFS_OP_READ, fs.hfid, base, st, nb, 0, 0, nullptr, 0, nullptr);
     if (r < 0) {
+      if (st >= 0) stage_free(c, st);
       atom_or_rel(&c->f_state[g], GFS_ST_ERROR);
       atom_and_rel(&c->f_state[g], ~GFS_ST_FILLING);
       atom_add_rel(&c->f_state[g], 0xFFFFFFFFu);
-      result = r == -ETIMEDOUT ? r : -EIO;
+      out.frame = r == -ETIMEDOUT ? r : -EIO;
+      out.fill = 0;
       break;
     }
-    st_rlx(&c->f_valid[g], (uint32_t)r);
-    atom_and_rel(&c->f_state[g], ~GFS_ST_FILLING);
+    out.stage = st;
+    out.nbytes = nb;
     ctr(c, GFS_C_MISS);
     ctr(c, GFS_C_RPC_READ);
     ctr(c, GFS_C_BYTES_H2D, nb);
-    result = g;
     break;
   }
   if (locked) {
     spin_unlock(lockp);
     ctr(c, GFS_C_LOCKED);
-  } else {
+  } else if (out.frame >= 0) {
     ctr(c, GFS_C_LOCKFREE);
   }
-  return result;
+  return out;
 }
 
-// ------------------------------------------------------------------ copies
-// Block-cooperative copy of n bytes. Frame reads bypass L1 (ld.global.cg):
-// a frame may have been refilled by DMA since this SM last cached it
-// (P:L693-696). 16-byte vectors with 4 loads in flight per thread when
-// src/dst are co-aligned; 4-byte or byte fallback otherwise.
-__device__ __forceinline__ void block_copy_from_frame(uint8_t* dst, const uint8_t* src, uint64_t n, int tid,
-                                                      int nthr) {
-  if (n == 0) return;
-  if ((((uintptr_t)src ^ (uintptr_t)dst) & 15) == 0) {
-    const uint64_t head = ((16 - ((uintptr_t)src & 15)) & 15) < n ? ((16 - ((uintptr_t)src & 15)) & 15) : n;
-    for (uint64_t i = tid; i < head; i += nthr) dst[i] = __ldcg(src + i);
-    const uint64_t nv = (n - head) >> 4;
-    const int4* s4 = (const int4*)(src + head);
-    int4* d4 = (int4*)(dst + head);
-    uint64_t i = tid;
-    const uint64_t stride = (uint64_t)nthr;
-    for (; i + 3 * stride < nv; i += 4 * stride) {
-      int4 a = __ldcg(s4 + i), b = __ldcg(s4 + i + stride), cc = __ldcg(s4 + i + 2 * stride),
-           d = __ldcg(s4 + i + 3 * stride);
-      d4[i] = a;
-      d4[i + stride] = b;
-      d4[i + 2 * stride] = cc;
-      d4[i + 3 * stride] = d;
+// Take references on pages [pb, pb + cnt) (cnt <= 32), all threads calling.
+// Lookups run one page per lane of warp 0 (parallel misses = parallel RPCs).
+// Pages this block installed are filled by the whole block: pulled from
+// staging over PCIe (O_RDONLY) — or, for O_GWRONCE, left FILLING with
+// sc.fill[i] = 1 for the caller (gwrite) to zero-fill/write. Busy pages are
+// retried after the block's own fills, so no block waits on another while it
+// holds an unfilled frame. Returns 0 with every sc.frame[i] held, or -errno
+// with none held.
+__device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, uint64_t pb, uint32_t cnt,
+                             bool first_done) {
+  const int tid = block_tid(), nthr = block_nthr();
+  const bool fast = !(c->flags & GFS_F_LOCKED_TRAVERSAL);
+  if (!first_done && tid < (int)cnt) sc.frame[tid] = kBusy;
+  const uint64_t t0 = now_ns();
+  uint32_t ns = 128;
+  for (int round = 0;; ++round) {
+    if (!(first_done && round == 0)) {
+      if (tid < (int)cnt && sc.frame[tid] == kBusy) {
+        int f = fast ? lookup_fast(c, fs, pb + tid) : -1;
+        if (f >= 0) {
+          sc.frame[tid] = f;
+          sc.fill[tid] = 0;
+          sc.stage[tid] = -1;
+        } else {
+          const Lk r = lookup_try(c, fs, pb + tid);
+          sc.frame[tid] = r.frame;
+          sc.fill[tid] = r.fill;
+          sc.stage[tid] = r.stage;
+          sc.nbytes[tid] = r.nbytes;
+        }
+      }
+      __syncthreads();
     }
-    for (; i < nv; i += stride) d4[i] = __ldcg(s4 + i);
-    const uint64_t done = head + (nv << 4);
-    for (uint64_t k = done + tid; k < n; k += nthr) dst[k] = __ldcg(src + k);
-  } else if ((((uintptr_t)src ^ (uintptr_t)dst) & 3) == 0) {
-    const uint64_t head = ((4 - ((uintptr_t)src & 3)) & 3) < n ? ((4 - ((uintptr_t)src & 3)) & 3) : n;
-    for (uint64_t i = tid; i < head; i += nthr) dst[i] = __ldcg(src + i);
-    const uint64_t nw = (n - head) >> 2;
-    const uint32_t* s4 = (const uint32_t*)(src + head);
-    uint32_t* d4 = (uint32_t*)(dst + head);
-    for (uint64_t i = tid; i < nw; i += nthr) d4[i] = __ldcg(s4 + i);
-    for (uint64_t k = head + (nw << 2) + tid; k < n; k += nthr) dst[k] = __ldcg(src + k);
-  } else {
-    for (uint64_t i = tid; i < n; i += nthr) dst[i] = __ldcg(src + i);
+    int err = 0;
+    bool busy = false, pull = false;
+    for (uint32_t i = 0; i < cnt; ++i) {
+      const int f = sc.frame[i];
+      if (f == kBusy) busy = true;
+      else if (f < 0) err = f;
+      else if (sc.fill[i] && sc.stage[i] >= 0) pull = true;
+    }
+    if (pull) {  // fill the frames this block installed: staging -> frame over PCIe
+      for (uint32_t i = 0; i < cnt; ++i)
+        if (sc.frame[i] >= 0 && sc.fill[i] && sc.stage[i] >= 0)
+          block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), stage_ptr(c, sc.stage[i]), sc.nbytes[i],
+                                      tid, nthr);
+      __threadfence();
+      __syncthreads();
+      if (tid < (int)cnt && sc.frame[tid] >= 0 && sc.fill[tid] && sc.stage[tid] >= 0) {
+        const uint32_t f = (uint32_t)sc.frame[tid];
+        stage_free(c, sc.stage[tid]);
+        sc.stage[tid] = -1;
+        sc.fill[tid] = 0;
+        st_rlx(&c->f_valid[f], sc.nbytes[tid]);
+        atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);  // publish the page
+      }
+    }
+    if (err) {
+      if (tid < (int)cnt && sc.frame[tid] >= 0) {
+        const uint32_t f = (uint32_t)sc.frame[tid];
+        if (sc.fill[tid]) {  // an installed O_GWRONCE page nobody wrote: give it back
+          st_rel64(&c->f_tag[f], GFS_TAG_NONE);
+          atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+        }
+        frame_release(c, f);
+      }
+      __syncthreads();
+      return err;
+    }
+    if (!busy) {
+      if (pull) __syncthreads();
+      return 0;
+    }
+    // still busy: back off and retry (the timeout decision is made by one
+    // thread and broadcast, so every thread takes the same path)
+    if (tid == 0) sc.busy = timed_out(c, t0) ? 1u : 0u;
+    if (tid < 32) __nanosleep(ns);
+    ns = ns < 2048 ? ns * 2 : 2048;
+    __syncthreads();
+    if (sc.busy) {
+      if (tid == 0) ctr(c, GFS_C_TIMEOUT);
+      if (tid < (int)cnt && sc.frame[tid] == kBusy) sc.frame[tid] = -ETIMEDOUT;  // error path next round
+      __syncthreads();
+    }
   }
-}
-
-// Block-cooperative copy into a frame (gwrite) — plain loads of user data.
-__device__ __forceinline__ void block_copy_to_frame(uint8_t* dst, const uint8_t* src, uint64_t n, int tid, int nthr) {
-  if (n == 0) return;
-  if ((((uintptr_t)src ^ (uintptr_t)dst) & 15) == 0) {
-    const uint64_t head = ((16 - ((uintptr_t)src & 15)) & 15) < n ? ((16 - ((uintptr_t)src & 15)) & 15) : n;
-    for (uint64_t i = tid; i < head; i += nthr) dst[i] = src[i];
-    const uint64_t nv = (n - head) >> 4;
-    const int4* s4 = (const int4*)(src + head);
-    int4* d4 = (int4*)(dst + head);
-    for (uint64_t i = tid; i < nv; i += nthr) d4[i] = s4[i];
-    for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = src[k];
-  } else {
-    for (uint64_t i = tid; i < n; i += nthr) dst[i] = src[i];
-  }
-}
-
-__device__ __forceinline__ void block_zero(uint8_t* dst, uint64_t n, int tid, int nthr) {
-  uint64_t i = tid;
-  const uint64_t head = ((16 - ((uintptr_t)dst & 15)) & 15) < n ? ((16 - ((uintptr_t)dst & 15)) & 15) : n;
-  for (; i < head; i += nthr) dst[i] = 0;
-  const uint64_t nv = (n - head) >> 4;
-  int4* d4 = (int4*)(dst + head);
-  for (uint64_t k = tid; k < nv; k += nthr) d4[k] = make_int4(0, 0, 0, 0);
-  for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = 0;
 }
 
 // ------------------------------------------------------------------ file table
@@ -735,15 +892,6 @@ __device__ __forceinline__ bool snap_fd(const gfs_ctx* c, int fd, FileSnap* s) {
   return true;
 }
 
-__device__ __forceinline__ uint64_t grid_id() {
-  uint64_t g;
-  asm volatile("mov.u64 %0, %%gridid;" : "=l"(g));
-  return g;
-}
-__device__ __forceinline__ uint32_t block_linear() {
-  return blockIdx.x + gridDim.x * (blockIdx.y + gridDim.y * blockIdx.z);
-}
-
 // Snapshot for gread: read-only files this block opened are served from the
 // block's cached snapshot (their entry cannot change while held open).
 __device__ __forceinline__ bool snap_fd_cached(const gfs_ctx* c, Scratch& sc, int fd, FileSnap* s) {
@@ -754,33 +902,45 @@ __device__ __forceinline__ bool snap_fd_cached(const gfs_ctx* c, Scratch& sc, in
   return snap_fd(c, fd, s);
 }
 
-// Write back every dirty, unreferenced page of the snapshot file in pages
-// [pb, pe), strided over the calling threads. Returns 0, -EBUSY (a dirty page
-// was mapped or in use, Tab.1), or a negative RPC error.
-__device__ int sync_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uint64_t pe, int tid, int nthr) {
+// Claim page p's frame for write-back if it is dirty and unreferenced.
+// Returns the frame (state EVICTING) or -1 (clean / absent), or -EBUSY.
+__device__ int claim_dirty(const gfs_ctx* c, const FileSnap& fs, uint64_t p) {
+  uint32_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
+  if (!slot) return -1;
+  const uint32_t s = ld_acq(slot);
+  if (!s) return -1;
+  const uint32_t f = s - 1;
+  const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
+  if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) return -1;
+  if (atom_cas(&c->f_state[f], 0u, GFS_ST_EVICTING) != 0u)
+    return (ld_acq64(&c->f_tag[f]) == want && ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) ? -EBUSY : -1;
+  if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) {
+    atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+    return -1;
+  }
+  return (int)f;
+}
+
+// Write back every dirty, unreferenced page of the snapshot file in [pb, pe)
+// from a single thread (used by the re-open path). Returns 0, -EBUSY (a dirty
+// page was mapped or in use, Tab.1), or a negative RPC error.
+__device__ int sync_pages_lane(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uint64_t pe) {
   int rc = 0;
-  for (uint64_t p = pb + tid; p < pe; p += nthr) {
-    uint32_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
-    if (!slot) continue;
-    const uint32_t s = ld_acq(slot);
-    if (!s) continue;
-    const uint32_t f = s - 1;
-    const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
-    if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) continue;
-    if (atom_cas(&c->f_state[f], 0u, GFS_ST_EVICTING) != 0u) {
-      if (ld_acq64(&c->f_tag[f]) == want && ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE && rc == 0) rc = -EBUSY;
+  for (uint64_t p = pb; p < pe; ++p) {
+    const int f = claim_dirty(c, fs, p);
+    if (f == -EBUSY) {
+      if (rc == 0) rc = -EBUSY;
       continue;
     }
-    if (ld_acq64(&c->f_tag[f]) == want) {
-      const int32_t r = frame_writeback(c, f, fs.hfid);
-      if (r < 0) rc = r;
-    }
+    if (f < 0) continue;
+    const int32_t r = frame_writeback_lane(c, (uint32_t)f, fs.hfid);
+    if (r < 0) rc = r;
     atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
   }
   return rc;
 }
 
-// Drop cached pages [pb, pe) of the snapshot file (gftruncate / invalidation).
+// Drop cached pages [pb, pe) of the snapshot file (gftruncate).
 __device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uint64_t pe, int tid, int nthr) {
   int rc = 0;
   for (uint64_t p = pb + tid; p < pe; p += nthr) {
@@ -819,7 +979,7 @@ __device__ __forceinline__ bool same_path(const gfs_ctx* c, const gfs_file* e, u
 __device__ int open_rpc_fill(const gfs_ctx* c, gfs_file* e, uint32_t fdx, uint32_t flags, uint32_t old_hfid_plus1,
                              gfs_rpc_resp* rs) {
   const char* sp = c->paths + (size_t)fdx * GFS_MAX_PATH;
-  const int32_t r = rpc_call(c, GFS_OP_OPEN, 0, 0, 0, 0, flags, old_hfid_plus1, sp, e->path_len, rs);
+  const int32_t r = rpc_call(c, GFS_OP_OPEN, 0, 0, -1, 0, flags, old_hfid_plus1, sp, e->path_len, rs);
   ctr(c, GFS_C_RPC_OPEN);
   if (r < 0) return r;
   if (rs->status < 0) return rs->status;
@@ -936,7 +1096,7 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
       old.hfid = e->hfid; old.oflags = e->oflags; old.size = e->size;
       if (old.oflags & GFS_O_GWRONCE) {  // never lose written data: sync before dropping
         const uint64_t np = (old.size + c->page_size - 1) >> c->page_shift;
-        int r = sync_pages(c, old, 0, np, 0, 1);
+        int r = sync_pages_lane(c, old, 0, np);
         if (r < 0 && r != -EBUSY) {
           sr_shift(e, GFS_FS_REOPENING, GFS_FS_CLOSED, -1);
           return r;
@@ -986,6 +1146,7 @@ __device__ int close_leader(const gfs_ctx* c, int fd) {
   return 0;  // no write-back
 }
 
+}  // namespace
 }  // namespace detail
 
 // ===================================================================== API
@@ -1040,9 +1201,10 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   const uint32_t shift = c->page_shift;
   const uint64_t P = c->page_size;
   const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
+  const bool fast = !(c->flags & GFS_F_LOCKED_TRAVERSAL);
   __syncthreads();  // the call is a barrier: earlier uses of dst by the block are complete
-  // Warp 0 alone: snapshot + clip, then the first batch of lookups (one page
-  // per lane). Other warps only touch `sc` after the next barrier.
+  // Warp 0 alone: snapshot + clip, then the first batch's fast-path lookups
+  // (one page per lane). Other warps only touch `sc` after the next barrier.
   if (tid < 32) {
     if (tid == 0) {
       FileSnap s;
@@ -1062,12 +1224,18 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
       const uint32_t cnt = (uint32_t)((q1 - q0 + 1) < B ? (q1 - q0 + 1) : B);
       if (tid < (int)cnt) {
         const FileSnap fs0 = sc.fs;
-        int f = (c->flags & GFS_F_LOCKED_TRAVERSAL) ? -1 : lookup_fast(c, fs0, q0 + tid);
+        int f = fast ? lookup_fast(c, fs0, q0 + tid) : -1;
         if (f < 0) {
-          uint32_t inst;
-          f = lookup_page(c, fs0, q0 + tid, &inst);
+          const Lk r = lookup_try(c, fs0, q0 + tid);
+          sc.frame[tid] = r.frame;
+          sc.fill[tid] = r.fill;
+          sc.stage[tid] = r.stage;
+          sc.nbytes[tid] = r.nbytes;
+        } else {
+          sc.frame[tid] = f;
+          sc.fill[tid] = 0;
+          sc.stage[tid] = -1;
         }
-        sc.frame[tid] = f;
       }
     }
   }
@@ -1078,40 +1246,24 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
   for (uint64_t pb = p0; pb <= p1; pb += B) {
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
-    if (pb != p0) {  // later batches: lookups by the first cnt threads
-      if (tid < (int)cnt) {
-        int f = (c->flags & GFS_F_LOCKED_TRAVERSAL) ? -1 : lookup_fast(c, fs, pb + tid);
-        if (f < 0) {
-          uint32_t inst;
-          f = lookup_page(c, fs, pb + tid, &inst);
-        }
-        sc.frame[tid] = f;
-      }
-      __syncthreads();
-    }
-    int err = 0;
-    for (uint32_t i = 0; i < cnt; ++i)
-      if (sc.frame[i] < 0) err = sc.frame[i];
-    if (!err) {
-      for (uint32_t i = 0; i < cnt; ++i) {
-        const uint64_t p = pb + i;
-        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
-        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-        uint8_t* d = (uint8_t*)dst + ((p << shift) + s - off);
-        const uint8_t* src = frame_ptr(c, (uint32_t)sc.frame[i]) + s;
-        block_copy_from_frame(d, src, e - s, tid, nthr);
-      }
+    const int err = acquire_batch(c, sc, fs, pb, cnt, pb == p0);
+    if (err) return err;
+    for (uint32_t i = 0; i < cnt; ++i) {
+      const uint64_t p = pb + i;
+      const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+      const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+      block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+                            e - s, tid, nthr);
     }
     __syncthreads();
-    if (tid < (int)cnt && sc.frame[tid] >= 0) frame_release(c, (uint32_t)sc.frame[tid]);
-    if (err) return err;
+    if (tid < (int)cnt) frame_release(c, (uint32_t)sc.frame[tid]);
   }
   return n;
 }
 
 // gwrite: pwrite semantics on an O_GWRONCE file.
 // New pages are zero-filled (never fetched); the dirty range and written byte
-// count are kept per frame; a fence makes the data visible to write-back DMA
+// count are kept per frame; a fence makes the data visible to write-back
 // (P:L577-582).
 __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, const void* src) {
   using namespace detail;
@@ -1140,44 +1292,32 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
   const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
   for (uint64_t pb = p0; pb <= p1; pb += B) {
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
+    const int err = acquire_batch(c, sc, fs, pb, cnt, false);
+    if (err) return err;
+    for (uint32_t i = 0; i < cnt; ++i) {
+      const uint64_t p = pb + i;
+      const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+      const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+      uint8_t* fp = frame_ptr(c, (uint32_t)sc.frame[i]);
+      if (sc.fill[i]) {  // pristine copy is zeros
+        block_zero(fp, s, tid, nthr);
+        block_zero(fp + e, P - e, tid, nthr);
+      }
+      block_copy_plain(fp + s, (const uint8_t*)src + ((p << shift) + s - off), e - s, tid, nthr);
+    }
+    __threadfence();
+    __syncthreads();
     if (tid < (int)cnt) {
-      uint32_t inst = 0;
-      sc.frame[tid] = lookup_page(c, fs, pb + tid, &inst);
-      sc.installed[tid] = inst;
-    }
-    __syncthreads();
-    int err = 0;
-    for (uint32_t i = 0; i < cnt; ++i)
-      if (sc.frame[i] < 0) err = sc.frame[i];
-    if (!err) {
-      for (uint32_t i = 0; i < cnt; ++i) {
-        const uint64_t p = pb + i;
-        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
-        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-        uint8_t* fp = frame_ptr(c, (uint32_t)sc.frame[i]);
-        if (sc.installed[i]) {  // pristine copy is zeros
-          block_zero(fp, s, tid, nthr);
-          block_zero(fp + e, P - e, tid, nthr);
-        }
-        block_copy_to_frame(fp + s, (const uint8_t*)src + ((p << shift) + s - off), e - s, tid, nthr);
-      }
-      __threadfence();
-    }
-    __syncthreads();
-    if (tid < (int)cnt && sc.frame[tid] >= 0) {
       const uint32_t f = (uint32_t)sc.frame[tid];
-      if (!err) {
-        const uint64_t p = pb + tid;
-        const uint32_t s = (uint32_t)(p == p0 ? (off & (P - 1)) : 0);
-        const uint32_t e = (uint32_t)(p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P);
-        atomicMin(&c->f_lo[f], s);
-        atomicMax(&c->f_hi[f], e);
-        atomicAdd(&c->f_written[f], e - s);
-      }
-      if (sc.installed[tid]) atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+      const uint64_t p = pb + tid;
+      const uint32_t s = (uint32_t)(p == p0 ? (off & (P - 1)) : 0);
+      const uint32_t e = (uint32_t)(p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P);
+      atomicMin(&c->f_lo[f], s);
+      atomicMax(&c->f_hi[f], e);
+      atomicAdd(&c->f_written[f], e - s);
+      if (sc.fill[tid]) atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
       frame_release_rel(c, f);
     }
-    if (err) return err;
   }
   if (tid == 0) atomicMax((unsigned long long*)&c->files[fd].size, (unsigned long long)(off + (uint64_t)n));
   __syncthreads();
@@ -1186,7 +1326,10 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
 
 // gfsync: synchronously write back all dirty pages of the file that are not
 // mapped or in use (Tab.1); on success the data is in the host page
-// cache. Returns -EBUSY if busy dirty pages were skipped.
+// cache. Block-cooperative: warp-0 lanes claim up to 32 dirty
+// pages, the block copies their dirty ranges into staging slots over PCIe,
+// then the lanes post the WRITE RPCs in parallel. Returns -EBUSY if busy
+// dirty pages were skipped.
 __device__ inline int gfsync(const gfs_ctx* c, int fd) {
   using namespace detail;
   Scratch& sc = scratch();
@@ -1207,8 +1350,54 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
   const FileSnap fs = sc.fs;
   if (fs.oflags & GFS_O_GWRONCE) {
     const uint64_t np = (fs.size + c->page_size - 1) >> c->page_shift;
-    const int r = sync_pages(c, fs, 0, np, tid, nthr);
-    if (r < 0) atomicMin(&sc.err, r);  // any error: -EIO etc. are < -EBUSY
+    const uint32_t B = nthr < 32 ? (uint32_t)nthr : 32u;
+    for (uint64_t pb = 0; pb < np; pb += B) {
+      const uint32_t cnt = (uint32_t)((np - pb) < B ? (np - pb) : B);
+      if (tid < (int)cnt) {
+        const int f = claim_dirty(c, fs, pb + tid);
+        sc.frame[tid] = f;
+        sc.stage[tid] = -1;
+        if (f == -EBUSY) atomicMin(&sc.err, -EBUSY);
+        if (f >= 0) {
+          sc.lo[tid] = ld_rlx(&c->f_lo[f]);
+          sc.hi[tid] = ld_rlx(&c->f_hi[f]);
+          const int st = stage_alloc(c);
+          sc.stage[tid] = st;
+          if (st < 0) {
+            atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+            sc.frame[tid] = -1;
+            atomicMin(&sc.err, st);
+          }
+        }
+      }
+      __syncthreads();
+      for (uint32_t i = 0; i < cnt; ++i)
+        if (sc.frame[i] >= 0)
+          block_copy_plain(stage_ptr(c, sc.stage[i]) + sc.lo[i], frame_ptr(c, (uint32_t)sc.frame[i]) + sc.lo[i],
+                           sc.hi[i] - sc.lo[i], tid, nthr);
+      __threadfence_system();
+      __syncthreads();
+      if (tid < (int)cnt && sc.frame[tid] >= 0) {
+        const uint32_t f = (uint32_t)sc.frame[tid];
+        const uint32_t lo = sc.lo[tid], hi = sc.hi[tid];
+        const uint32_t wr = ld_rlx(&c->f_written[f]);
+        const int32_t r = rpc_call(c, GFS_OP_WRITE, fs.hfid, ((pb + tid) << c->page_shift) + lo, sc.stage[tid],
+                                   hi - lo, wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, nullptr);
+        stage_free(c, sc.stage[tid]);
+        if (r < 0) {
+          atomicMin(&sc.err, r);
+        } else {
+          st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
+          st_rlx(&c->f_hi[f], 0);
+          st_rlx(&c->f_written[f], 0);
+          ctr(c, GFS_C_WRITEBACK);
+          ctr(c, GFS_C_RPC_WRITE);
+          ctr(c, GFS_C_BYTES_D2H, hi - lo);
+        }
+        atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+      }
+      __syncthreads();
+    }
   }
   __syncthreads();
   return sc.err;
@@ -1231,24 +1420,32 @@ __device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int pr
     FileSnap s;
     sc.ptr = nullptr;
     sc.aux = 0;
-    if (!snap_fd(c, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
+    sc.ret = 0;
+    if (!snap_fd_cached(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
       sc.aux = -EBADF;
     } else if (off < s.size && len > 0) {
-      uint32_t inst;
-      const int f = lookup_page(c, s, off >> c->page_shift, &inst);
-      if (f < 0) {
-        sc.aux = f;
+      sc.fs = s;
+      sc.ret = 1;
+    }
+  }
+  __syncthreads();
+  if (sc.ret == 1) {
+    const FileSnap fs = sc.fs;
+    const int err = acquire_batch(c, sc, fs, off >> c->page_shift, 1, false);
+    if (tid == 0) {
+      if (err) {
+        sc.aux = err;
       } else {
         const uint64_t in = off & (c->page_size - 1);
         uint64_t m = c->page_size - in;
         if (len < m) m = len;
-        if (s.size - off < m) m = s.size - off;
-        sc.ptr = frame_ptr(c, (uint32_t)f) + in;
+        if (fs.size - off < m) m = fs.size - off;
+        sc.ptr = frame_ptr(c, (uint32_t)sc.frame[0]) + in;
         sc.aux = (int64_t)m;
       }
     }
+    __syncthreads();
   }
-  __syncthreads();
   if (mapped_len) *mapped_len = sc.aux > 0 ? (uint64_t)sc.aux : 0;
   return sc.ptr;
 }
@@ -1287,7 +1484,7 @@ __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
     } else {
       sc.fs = s;
       sc.err = 0;
-      const int32_t r = rpc_call(c, GFS_OP_TRUNC, s.hfid, 0, 0, 0, 0, size, nullptr, 0, nullptr);
+      const int32_t r = rpc_call(c, GFS_OP_TRUNC, s.hfid, 0, -1, 0, 0, size, nullptr, 0, nullptr);
       sc.ret = r < 0 ? r : 0;
       if (r >= 0) st_rlx64((uint64_t*)&c->files[fd].size, size);
     }

@@ -93,7 +93,7 @@ typedef struct gfs_rpc_req { /* one 64-byte ring slot in pinned host memory */
   uint32_t flags;
   uint64_t arg;
   uint32_t path_len;
-  uint32_t pad0;
+  uint32_t stage;    /* READ/WRITE: staging slot holding the data (host-mapped pinned memory) */
   uint64_t pad1;
   uint64_t seq;      /* = ticket + 1; written LAST with st.release.sys */
 } gfs_rpc_req;
@@ -108,7 +108,10 @@ typedef struct gfs_rpc_resp { /* OPEN reply, host-written before completion */
   uint64_t pad[2];
 } gfs_rpc_resp;
 
-/* completion word (device memory): ((ticket + 1) << 32) | (uint32_t)result */
+/* completion word (pinned, mapped host memory; host store-release, GPU
+ * ld.acquire.sys): ((ticket + 1) << 32) | (uint32_t)result. The daemon makes
+ * no CUDA call per RPC: data moves through host-mapped staging slots that the
+ * GPU itself reads (fill) or writes (write-back) over PCIe. */
 
 /* ---- counters (Table 2 analogue + RPC accounting) --------------------- */
 enum {
@@ -136,6 +139,8 @@ enum {
   GFS_C_GWRITE_CALLS,
   GFS_C_NODES,          /* radix nodes allocated */
   GFS_C_RING_WAIT,      /* ring slot was busy on post */
+  GFS_C_BUSY,           /* lookups that found the page being filled/evicted by another block */
+  GFS_C_STAGE_WAIT,     /* staging slot allocation had to wait */
   GFS_C_NCOUNTERS
 };
 
@@ -173,9 +178,15 @@ typedef struct gfs_ctx {
   gfs_rpc_req* ring;   /* device-mapped pointer to pinned host ring */
   gfs_rpc_resp* resp;  /* device-mapped pointer to pinned host responses */
   char* ring_paths;    /* device-mapped, ring_slots * GFS_MAX_PATH */
-  uint64_t* cpl;       /* device memory completion words */
+  uint64_t* cpl;       /* device-mapped pinned host memory: completion words */
   uint64_t* ack;       /* device memory: slot released by its client */
   unsigned long long* ring_tail;
+  /* staging: pinned host slots of page_size bytes, device-mapped */
+  uint8_t* staging;
+  uint32_t staging_slots;
+  uint32_t staging_words;  /* bitmap words */
+  uint32_t* staging_bits;  /* device memory: 1 = slot in use */
+  uint32_t pad_staging;
   /* config */
   uint32_t flags;
   uint32_t max_batch;

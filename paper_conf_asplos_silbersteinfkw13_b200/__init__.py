@@ -18,7 +18,7 @@ LIB_PATH = os.path.join(_PKG, "libgpufs.so")
 COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", "writeback", "rpc",
             "rpc_open", "rpc_read", "rpc_write", "bytes_h2d", "bytes_d2h", "open_fast", "reopen_valid",
             "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
-            "ring_wait"]
+            "ring_wait", "busy", "stage_wait"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
                  "errors", "merges"]
 
@@ -38,9 +38,18 @@ class gfs_config(ctypes.Structure):
     _fields_ = [("device", ctypes.c_int), ("cache_bytes", ctypes.c_uint64), ("page_size", ctypes.c_uint32),
                 ("ring_slots", ctypes.c_uint32), ("daemon_threads", ctypes.c_uint32),
                 ("max_files", ctypes.c_uint32), ("max_nodes", ctypes.c_uint32), ("max_batch", ctypes.c_uint32),
-                ("flags", ctypes.c_uint32), ("pad", ctypes.c_uint32), ("timeout_ms", ctypes.c_uint64),
+                ("flags", ctypes.c_uint32), ("staging_slots", ctypes.c_uint32), ("timeout_ms", ctypes.c_uint64),
                 ("frame_pool", ctypes.c_void_p)]
 
+
+class gfs_grep_params(ctypes.Structure):
+    _fields_ = [("max_files", ctypes.c_uint32), ("max_words", ctypes.c_uint32), ("list_cap", ctypes.c_uint64),
+                ("pair_cap", ctypes.c_uint64), ("hit_cap", ctypes.c_uint64), ("chunk", ctypes.c_uint32),
+                ("grid", ctypes.c_uint32), ("block", ctypes.c_uint32), ("keep_open", ctypes.c_uint32)]
+
+
+GREP_SUMMARY = ["nrecords", "nhits", "digest_sum", "digest_xor", "nfiles", "nwords", "bytes", "err",
+                "nhits_listed", "nitems"]
 
 _lib = None
 
@@ -70,6 +79,8 @@ def lib():
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32], I),
             "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
+            "gfs_grep_work_bytes": ([ctypes.POINTER(gfs_grep_params)], U64),
+            "gfs_grep": ([P, P, CS, CS, ctypes.POINTER(gfs_grep_params), P, P, U64, P, P, P], I),
         }
         for name, (args, res) in sig.items():
             fn = getattr(L, name)
@@ -136,7 +147,7 @@ def gfs_info(h: int) -> dict:
     a = (ctypes.c_uint64 * 9)()
     _ck(lib().gfs_info(h, a, 9), "gfs_info")
     return dict(zip(["page_size", "nframes", "max_files", "max_nodes", "ring_slots", "daemon_threads",
-                     "stream_write_value64", "host_next_ticket", "device_ring_tail"], (int(x) for x in a)))
+                     "staging_slots", "host_next_ticket", "device_ring_tail"], (int(x) for x in a)))
 
 
 # ------------------------------------------------------------------ launchers
@@ -162,6 +173,16 @@ def gfs_run_gwrite(h, stream, path, ncalls, d_off, d_len, d_srcoff, d_src, d_ret
 
 def gfs_run_fileop(h, stream, path, flags, op, arg, d_ret):
     return _ck(lib().gfs_run_fileop(h, stream, _b(path), flags, op, arg, d_ret), "gfs_run_fileop")
+
+
+def gfs_grep_work_bytes(p: gfs_grep_params) -> int:
+    return int(lib().gfs_grep_work_bytes(ctypes.byref(p)))
+
+
+def gfs_grep(h, stream, dict_path, list_path, p: gfs_grep_params, d_work, d_rec, rec_cap, d_totals, d_hits,
+             d_summary):
+    return _ck(lib().gfs_grep(h, stream, _b(dict_path), _b(list_path), ctypes.byref(p), d_work, d_rec, rec_cap,
+                              d_totals, d_hits, d_summary), "gfs_grep")
 
 
 from . import build  # noqa: E402,F401

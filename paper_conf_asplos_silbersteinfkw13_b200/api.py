@@ -24,14 +24,15 @@ class GpuFS:
     """One GPU buffer cache + its host daemon (gfs_init + gfs_daemon)."""
 
     def __init__(self, cache_bytes=1 << 30, page_size=64 << 10, device=0, daemon_threads=8, ring_slots=4096,
-                 max_files=4096, max_nodes=0, max_batch=32, flags=0, timeout_ms=60000):
+                 max_files=4096, max_nodes=0, max_batch=32, flags=0, timeout_ms=60000, staging_slots=0):
         torch = _torch()
         torch.cuda.set_device(device)
         self.device = device
         self.page_size = page_size
         cfg = gfs_config_default(device=device, cache_bytes=cache_bytes, page_size=page_size,
                                  daemon_threads=daemon_threads, ring_slots=ring_slots, max_files=max_files,
-                                 max_nodes=max_nodes, max_batch=max_batch, flags=flags, timeout_ms=timeout_ms)
+                                 max_nodes=max_nodes, max_batch=max_batch, flags=flags, timeout_ms=timeout_ms,
+                                 staging_slots=staging_slots)
         self.h = gfs_init(cfg)
         gfs_daemon(self.h, DAEMON_SPAWN)
 
@@ -170,6 +171,61 @@ class GpuFS:
         gfs_run_fileop(self.h, sp, path, flags, code, arg, d_ret.data_ptr())
         s.synchronize()
         return int(d_ret.item())
+
+    # grep -w ------------------------------------------------------------------
+    def grep(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
+             pair_cap=1 << 22, hit_cap=None, stream=None, sync=True, state=None):
+        """grep -w. Returns a dict with records (n,3) sorted by (file, word),
+        totals, digest (sum, xor, nhits), hits (n,3) sorted by (file, offset, word) if requested.
+
+        Capacities come from file metadata (stat), never from file contents: the
+        contents are read on the GPU through gopen/gread."""
+        import os
+        torch = _torch()
+        from . import GREP_SUMMARY, gfs_grep, gfs_grep_params, gfs_grep_work_bytes
+        dev = f"cuda:{self.device}"
+        if state is None:
+            nwords = max(1, os.path.getsize(dict_path) // 32)
+            lbytes = os.path.getsize(list_path)
+            p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
+                                pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 2 * 148, block=block,
+                                keep_open=1 if keep_open else 0)
+            if hits:
+                p.hit_cap = hit_cap if hit_cap is not None else 1 << 22
+            work = torch.empty(gfs_grep_work_bytes(p), dtype=torch.uint8, device=dev)
+            rec = torch.empty(3 * p.pair_cap, dtype=torch.int32, device=dev)
+            totals = torch.empty(nwords, dtype=torch.int64, device=dev)
+            d_hits = torch.empty(2 * max(p.hit_cap, 1), dtype=torch.int64, device=dev) if hits else None
+            summ = torch.zeros(10, dtype=torch.int64, device=dev)
+            state = dict(p=p, work=work, rec=rec, totals=totals, hits=d_hits, summary=summ)
+        p = state["p"]
+        s, sp = self._stream(stream)
+        gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
+                 p.pair_cap, state["totals"].data_ptr(),
+                 state["hits"].data_ptr() if state["hits"] is not None else None, state["summary"].data_ptr())
+        if not sync:
+            return state
+        s.synchronize()
+        summ = dict(zip(GREP_SUMMARY, (int(x) for x in state["summary"].cpu().numpy())))
+        if summ["err"] == -28 and pair_cap < (1 << 30):  # -ENOSPC: (file, word) table too small
+            return self.grep(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap * 4, hit_cap,
+                             stream, sync)
+        out = {"summary": summ}
+        nrec = min(summ["nrecords"], p.pair_cap)
+        r = state["rec"][:3 * nrec].view(nrec, 3).cpu().numpy().astype(np.uint64)
+        order = np.lexsort((r[:, 1], r[:, 0])) if nrec else np.zeros(0, np.int64)
+        out["records"] = r[order]
+        out["totals"] = state["totals"][:summ["nwords"]].cpu().numpy().astype(np.uint64)
+        out["digest"] = (summ["digest_sum"] & ((1 << 64) - 1), summ["digest_xor"] & ((1 << 64) - 1), summ["nhits"])
+        if hits:
+            nl = min(summ["nhits_listed"], p.hit_cap)
+            hv = state["hits"][:2 * nl].view(nl, 2).cpu().numpy().view(np.uint64)
+            hh = np.stack([hv[:, 0] >> np.uint64(32), hv[:, 1], hv[:, 0] & np.uint64(0xFFFFFFFF)], axis=1) \
+                if nl else np.zeros((0, 3), np.uint64)
+            order = np.lexsort((hh[:, 2], hh[:, 1], hh[:, 0])) if nl else np.zeros(0, np.int64)
+            out["hits"] = hh[order]
+        out["state"] = state
+        return out
 
     def pin(self, path, flags=0) -> int:
         """Open `path` and keep it open across launches (later gopen calls need no RPC)."""

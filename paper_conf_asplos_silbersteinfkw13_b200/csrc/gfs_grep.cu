@@ -1,0 +1,618 @@
+// gfs_grep.cu — exact whole-word string search (grep -w) over many files,
+// built on the GPUfs device API (§5.2.2).
+//
+// Problem statement: for each dictionary word, how many times
+// and in which files it appears. Dictionary: one word per 32-byte slot
+// (P:L1264-1266). The list of input files is itself read from a file
+// (P:L1266-1267). Every file byte reaches the kernels through gopen/gread.
+//
+// The paper assigns one dictionary word per thread and brute-forces every
+// position. Here the result is the same (pinned
+// against the brute-force oracle) but the work is proportional to the corpus:
+//   k_grep_dict  gread the dictionary, validate slots, build an open-addressing
+//                hash table (L2-resident) keyed by a 64-bit token hash;
+//   k_grep_list  gread the file list and split it into absolute paths;
+//   k_grep_open  gopen every file once (first gopen goes to the host,
+//                P:L370-372), record fd and size, cut files into work items;
+//   k_grep_plan  exclusive scan of per-file item counts;
+//   k_grep_scan  persistent blocks pull items (file, chunk): gread the chunk
+//                plus a halo into shared memory, find token starts
+//                (W(t[i]) and not W(t[i-1])), hash + probe each token of
+//                <= 32 bytes, count matches per item in shared memory, flush
+//                (file, word) counts into a global table and word totals;
+//   k_grep_close gclose every file (unless kept open for warm re-runs);
+//   k_grep_compact  emit unique (file, word, count) records.
+// Word bytes are [A-Za-z0-9_] (GNU grep -w under LC_ALL=C, R10).
+#include <cuda_runtime.h>
+#include <errno.h>
+#include <stdint.h>
+#include <stdio.h>
+#include <string.h>
+
+#include "gpufs.h"
+#include "gpufs_device.cuh"
+
+#define GFS_API extern "C" __attribute__((visibility("default")))
+
+using namespace gfs;
+
+namespace {
+
+constexpr uint32_t kMaxPath = GFS_MAX_PATH;
+constexpr uint32_t kHalo = 48;      // bytes after the chunk: a token starting inside may run 33 bytes
+constexpr uint32_t kPre = 16;       // bytes before the chunk (one needed for the boundary test)
+constexpr uint32_t kCountSlots = 2048;
+constexpr uint64_t kPairEmpty = ~0ull;
+
+struct GrepWork {
+  // dictionary
+  uint8_t* dict;          // max_words * 32
+  uint64_t* table;        // dict hash table: (fp32 << 32) | (len << 26) | (k + 1); 0 = empty
+  uint32_t table_mask;
+  uint32_t* dup_head;     // per primary word: first duplicate + 1
+  uint32_t* dup_next;     // per word: next duplicate + 1
+  // file list
+  uint8_t* list;          // list_cap bytes
+  char* paths;            // max_files * kMaxPath
+  uint32_t* path_len;
+  int32_t* fd;
+  uint64_t* size;
+  uint64_t* item_base;    // max_files + 1
+  // (file, word) -> count table
+  uint64_t* pair_key;
+  uint64_t* pair_cnt;
+  uint64_t pair_mask;
+  // counters
+  unsigned long long* vars;  // see V_*
+};
+enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS, V_DSUM, V_DXOR, V_NLISTED,
+       V_NEXTF, V_NVARS };
+
+__device__ __forceinline__ bool is_word(uint32_t ch) {
+  return (ch - 'a' < 26u) || (ch - 'A' < 26u) || (ch - '0' < 10u) || ch == '_';
+}
+
+__device__ __forceinline__ uint64_t tok_hash(const uint8_t* p, uint32_t n) {
+  uint64_t h = 0xcbf29ce484222325ull;
+  for (uint32_t i = 0; i < n; ++i) h = (h ^ p[i]) * 0x100000001b3ull;
+  h ^= h >> 29;
+  h *= 0xbf58476d1ce4e5b9ull;
+  return h ^ (h >> 32);
+}
+
+__device__ __forceinline__ uint64_t splitmix64(uint64_t x) {
+  uint64_t z = x + 0x9E3779B97F4A7C15ull;
+  z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+  z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+  return z ^ (z >> 31);
+}
+
+// Order-independent digest term of one hit (file f, byte offset off, word k).
+__device__ __forceinline__ uint64_t hit_mix(uint64_t f, uint64_t off, uint64_t k) {
+  return splitmix64(splitmix64(splitmix64(f) + off) + k);
+}
+
+__device__ __forceinline__ void set_err(GrepWork& w, long long e) { atomicMin((long long*)&w.vars[V_ERR], e); }
+
+// --------------------------------------------------------------- dictionary
+__global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w, uint32_t max_words) {
+  const int tid = threadIdx.x;
+  const int fd = gopen(c, dict_path, GFS_O_RDONLY);
+  if (fd < 0) {
+    if (tid == 0 && blockIdx.x == 0) set_err(w, fd);
+    return;
+  }
+  const int64_t size = gfstat_size(c, fd);
+  if (size % 32 != 0 || size / 32 > (int64_t)max_words) {
+    if (tid == 0 && blockIdx.x == 0) set_err(w, size % 32 ? -EINVAL : -ENOSPC);
+    gclose(c, fd);
+    return;
+  }
+  const uint32_t N = (uint32_t)(size / 32);
+  if (blockIdx.x == 0 && tid == 0) w.vars[V_NWORDS] = N;
+  // each block reads a contiguous slice of slots, then inserts those words
+  const uint32_t per = (N + gridDim.x - 1) / gridDim.x;
+  const uint32_t k0 = blockIdx.x * per, k1 = min(N, k0 + per);
+  if (k0 < k1) {
+    const int64_t r = gread(c, fd, (uint64_t)k0 * 32, (uint64_t)(k1 - k0) * 32, w.dict + (size_t)k0 * 32);
+    __threadfence();  // this block's dictionary bytes are visible before its table entries
+    if (r != (int64_t)(k1 - k0) * 32) {
+      if (tid == 0) set_err(w, r < 0 ? r : -EIO);
+    } else {
+      for (uint32_t k = k0 + tid; k < k1; k += blockDim.x) {
+        const uint8_t* s = w.dict + (size_t)k * 32;
+        uint32_t n = 0;
+        while (n < 32 && s[n]) ++n;
+        bool ok = n > 0;
+        for (uint32_t i = 0; i < n; ++i) ok &= is_word(s[i]);
+        if (!ok) {  // empty slot or non-word byte (R13)
+          set_err(w, -EINVAL);
+          continue;
+        }
+        const uint64_t h = tok_hash(s, n);
+        const uint64_t ent = ((h >> 32) << 32) | ((uint64_t)n << 26) | (k + 1);
+        uint32_t slot = (uint32_t)h & w.table_mask;
+        for (uint32_t probe = 0; probe <= w.table_mask; ++probe, slot = (slot + 1) & w.table_mask) {
+          unsigned long long cur = atomicCAS((unsigned long long*)&w.table[slot], 0ull, (unsigned long long)ent);
+          if (cur == 0) break;
+          if ((cur >> 26) == (ent >> 26)) {  // same fingerprint and length: same word?
+            const uint32_t kp = (uint32_t)(cur & ((1u << 26) - 1)) - 1;
+            const uint8_t* t = w.dict + (size_t)kp * 32;
+            bool same = true;
+            for (uint32_t i = 0; i < n; ++i) same &= t[i] == s[i];
+            if (same) {  // duplicate dictionary word: chain it behind kp
+              w.dup_next[k] = atomicExch(&w.dup_head[kp], k + 1);
+              break;
+            }
+          }
+        }
+      }
+    }
+  }
+  gclose(c, fd);
+}
+
+// --------------------------------------------------------------- file list
+// One block: read the list, find non-empty lines, emit absolute paths.
+__global__ void k_grep_list(const gfs_ctx* c, const char* list_path, const char* dir, uint32_t dir_len,
+                            GrepWork w, uint64_t list_cap, uint32_t max_files) {
+  __shared__ uint32_t warp_tot[32];
+  __shared__ uint32_t base_s;
+  const int tid = threadIdx.x, nthr = blockDim.x;
+  const int fd = gopen(c, list_path, GFS_O_RDONLY);
+  if (fd < 0) {
+    if (tid == 0) set_err(w, fd);
+    return;
+  }
+  const int64_t size = gfstat_size(c, fd);
+  if (size > (int64_t)list_cap) {
+    if (tid == 0) set_err(w, -ENOSPC);
+    gclose(c, fd);
+    return;
+  }
+  const int64_t r = gread(c, fd, 0, (uint64_t)size, w.list);
+  gclose(c, fd);
+  if (r != size) {
+    if (tid == 0) set_err(w, r < 0 ? r : -EIO);
+    return;
+  }
+  if (tid == 0) base_s = 0;
+  __syncthreads();
+  const uint8_t* L = w.list;
+  // tiles of nthr bytes: thread i checks byte (tile + i) for a line start
+  for (int64_t t0 = 0; t0 < size; t0 += nthr) {
+    const int64_t i = t0 + tid;
+    bool start = false;
+    if (i < size) start = L[i] != '\n' && (i == 0 || L[i - 1] == '\n');
+    const uint32_t bal = __ballot_sync(0xFFFFFFFFu, start);
+    const int lane = tid & 31, wid = tid >> 5;
+    if (lane == 0) warp_tot[wid] = __popc(bal);
+    __syncthreads();
+    uint32_t before = base_s;
+    for (int q = 0; q < wid; ++q) before += warp_tot[q];
+    before += __popc(bal & ((1u << lane) - 1));
+    if (start) {
+      const uint32_t k = before;
+      if (k < max_files) {
+        uint32_t n = 0;
+        while (i + n < size && L[i + n] != '\n') ++n;
+        char* dst = w.paths + (size_t)k * kMaxPath;
+        uint32_t o = 0;
+        if (L[i] != '/') {  // relative to the list file's directory (R15)
+          for (uint32_t q = 0; q < dir_len && o < kMaxPath - 1; ++q) dst[o++] = dir[q];
+          if (o < kMaxPath - 1) dst[o++] = '/';
+        }
+        if (o + n >= kMaxPath) {
+          set_err(w, -ENAMETOOLONG);
+          n = 0;
+        }
+        for (uint32_t q = 0; q < n; ++q) dst[o + q] = (char)L[i + q];
+        dst[o + n] = 0;
+        w.path_len[k] = o + n;
+      } else {
+        set_err(w, -ENOSPC);
+      }
+    }
+    __syncthreads();
+    if (tid == 0) {
+      uint32_t tot = 0;
+      for (int q = 0; q < (nthr + 31) / 32; ++q) tot += warp_tot[q];
+      base_s += tot;
+    }
+    __syncthreads();
+  }
+  if (tid == 0) w.vars[V_NFILES] = base_s < max_files ? base_s : max_files;
+}
+
+// --------------------------------------------------------------- open files
+__global__ void k_grep_open(const gfs_ctx* c, GrepWork w, uint32_t chunk) {
+  __shared__ uint32_t f_s;
+  const int tid = threadIdx.x;
+  const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
+  for (;;) {
+    if (tid == 0) f_s = (uint32_t)atomicAdd(&w.vars[V_NEXTF], 1ull);
+    __syncthreads();
+    const uint32_t f = f_s;
+    if (f >= nfiles) break;
+    const int fd = gopen(c, w.paths + (size_t)f * kMaxPath, GFS_O_RDONLY);
+    const int64_t sz = fd >= 0 ? gfstat_size(c, fd) : fd;
+    if (tid == 0) {
+      w.fd[f] = fd;
+      if (sz < 0) {
+        set_err(w, sz);
+        w.size[f] = 0;
+        w.item_base[f] = 0;
+      } else {
+        w.size[f] = (uint64_t)sz;
+        w.item_base[f] = ((uint64_t)sz + chunk - 1) / chunk;  // item count; scanned later
+        atomicAdd(&w.vars[V_BYTES], (unsigned long long)sz);
+      }
+    }
+    __syncthreads();
+  }
+}
+
+// exclusive scan of item counts -> item_base, one block
+__global__ void k_grep_plan(GrepWork w) {
+  __shared__ uint64_t part[1024];
+  const int tid = threadIdx.x, nthr = blockDim.x;
+  const uint32_t n = (uint32_t)w.vars[V_NFILES];
+  const uint32_t per = (n + nthr - 1) / nthr;
+  const uint32_t a = tid * per, b = min(n, a + per);
+  uint64_t s = 0;
+  for (uint32_t i = a; i < b; ++i) s += w.item_base[i];
+  part[tid] = s;
+  __syncthreads();
+  if (tid == 0) {
+    uint64_t run = 0;
+    for (int q = 0; q < nthr; ++q) {
+      const uint64_t v = part[q];
+      part[q] = run;
+      run += v;
+    }
+    w.vars[V_NITEMS] = run;
+    w.item_base[n] = run;
+  }
+  __syncthreads();
+  uint64_t run = part[tid];
+  for (uint32_t i = a; i < b; ++i) {
+    const uint64_t v = w.item_base[i];
+    w.item_base[i] = run;
+    run += v;
+  }
+}
+
+// --------------------------------------------------------------- scan
+__device__ __forceinline__ void pair_add(GrepWork& w, uint32_t f, uint32_t k, uint64_t cnt) {
+  const uint64_t key = ((uint64_t)f << 32) | k;
+  uint64_t slot = splitmix64(key) & w.pair_mask;
+  for (uint64_t probe = 0; probe <= w.pair_mask; ++probe, slot = (slot + 1) & w.pair_mask) {
+    unsigned long long cur = atomicCAS((unsigned long long*)&w.pair_key[slot], (unsigned long long)kPairEmpty,
+                                       (unsigned long long)key);
+    if (cur == kPairEmpty || cur == key) {
+      atomicAdd((unsigned long long*)&w.pair_cnt[slot], (unsigned long long)cnt);
+      return;
+    }
+  }
+  set_err(w, -ENOSPC);
+}
+
+__global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w, uint32_t chunk, uint64_t* hits,
+                                                   uint64_t hit_cap) {
+  extern __shared__ __align__(16) uint8_t sm[];
+  uint8_t* buf = sm;                                               // chunk + kPre + kHalo
+  uint32_t* ckey = (uint32_t*)(sm + ((chunk + kPre + kHalo + 15) & ~15u));  // word + 1
+  uint32_t* ccnt = ckey + kCountSlots;
+  __shared__ uint64_t item_s;
+  const int tid = threadIdx.x, nthr = blockDim.x;
+  const uint64_t nitems = w.vars[V_NITEMS];
+  const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
+  uint64_t dsum = 0, dxor = 0, nh = 0;
+  for (uint32_t i = tid; i < kCountSlots; i += nthr) {  // dynamic smem is not cleared between launches
+    ckey[i] = 0;
+    ccnt[i] = 0;
+  }
+  for (;;) {
+    __syncthreads();
+    if (tid == 0) item_s = atomicAdd(&w.vars[V_NEXT], 1ull);
+    __syncthreads();
+    const uint64_t item = item_s;
+    if (item >= nitems) break;
+    // file of this item: last f with item_base[f] <= item
+    uint32_t lo = 0, hi = nfiles;
+    while (hi - lo > 1) {
+      const uint32_t mid = (lo + hi) >> 1;
+      if (w.item_base[mid] <= item) lo = mid; else hi = mid;
+    }
+    const uint32_t f = lo;
+    const int fd = w.fd[f];
+    const uint64_t size = w.size[f];
+    const uint64_t s = (item - w.item_base[f]) * chunk;
+    const uint64_t e = min(size, s + chunk);
+    const uint64_t ws = s >= kPre ? s - kPre : 0;
+    const uint64_t we = min(size, e + kHalo);
+    const int64_t r = gread(c, fd, ws, we - ws, buf);
+    if (r != (int64_t)(we - ws)) {
+      if (tid == 0) set_err(w, r < 0 ? r : -EIO);
+      continue;
+    }
+    // positions [s, e) in file coordinates map to buf[pos - ws]
+    const uint32_t n_here = (uint32_t)(e - s);
+    for (uint32_t q = tid; q < n_here; q += nthr) {
+      const uint64_t pos = s + q;
+      const uint32_t bi = (uint32_t)(pos - ws);
+      const uint32_t ch = buf[bi];
+      if (!is_word(ch)) continue;
+      if (pos > 0 && is_word(buf[bi - 1])) continue;
+      uint32_t L = 1;
+      while (L <= 32 && pos + L < size && is_word(buf[bi + L])) ++L;
+      if (L > 32) continue;  // tokens longer than any dictionary word never match
+      const uint64_t h = tok_hash(buf + bi, L);
+      uint32_t slot = (uint32_t)h & w.table_mask;
+      const uint64_t want = ((h >> 32) << 32) | ((uint64_t)L << 26);
+      for (;;) {
+        const uint64_t ent = __ldg((const unsigned long long*)&w.table[slot]);
+        if (ent == 0) break;
+        if ((ent >> 26) == (want >> 26)) {
+          const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
+          const uint8_t* t = w.dict + (size_t)kp * 32;
+          bool same = true;
+          for (uint32_t i = 0; i < L; ++i) same &= t[i] == buf[bi + i];
+          if (same) {
+            uint32_t k = kp;
+            for (;;) {  // the word and its duplicates (each index counts, R14)
+              // per-item count in shared memory; spill to the global table if full
+              uint32_t cs = (k * 2654435761u) & (kCountSlots - 1);
+              bool done = false;
+              for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & (kCountSlots - 1)) {
+                const uint32_t prev = atomicCAS(&ckey[cs], 0u, k + 1);
+                if (prev == 0 || prev == k + 1) {
+                  atomicAdd(&ccnt[cs], 1u);
+                  done = true;
+                  break;
+                }
+              }
+              if (!done) pair_add(w, f, k, 1);
+              const uint64_t m = hit_mix(f, pos, k);
+              dsum += m;
+              dxor ^= m;
+              ++nh;
+              if (hits) {
+                const unsigned long long idx = atomicAdd(&w.vars[V_NLISTED], 1ull);
+                if (idx < hit_cap) {
+                  hits[2 * idx] = ((uint64_t)f << 32) | k;
+                  hits[2 * idx + 1] = pos;
+                }
+              }
+              const uint32_t nx = w.dup_head[k] ? w.dup_head[k] : 0;
+              if (k == kp) {
+                if (!nx) break;
+                k = nx - 1;
+              } else {
+                const uint32_t nn = w.dup_next[k];
+                if (!nn) break;
+                k = nn - 1;
+              }
+            }
+            break;
+          }
+        }
+        slot = (slot + 1) & w.table_mask;
+      }
+    }
+    __syncthreads();
+    // flush this item's counts: (file, word) table and word totals
+    for (uint32_t i = tid; i < kCountSlots; i += nthr) {
+      const uint32_t kk = ckey[i];
+      if (kk) {
+        const uint32_t cnt = ccnt[i];
+        pair_add(w, f, kk - 1, cnt);
+        ckey[i] = 0;
+        ccnt[i] = 0;
+      }
+    }
+  }
+  // block-level digest reduction
+  for (int o = 16; o; o >>= 1) {
+    dsum += __shfl_xor_sync(0xFFFFFFFFu, dsum, o);
+    dxor ^= __shfl_xor_sync(0xFFFFFFFFu, dxor, o);
+    nh += __shfl_xor_sync(0xFFFFFFFFu, nh, o);
+  }
+  if ((tid & 31) == 0) {
+    atomicAdd(&w.vars[V_DSUM], (unsigned long long)dsum);
+    atomicXor(&w.vars[V_DXOR], (unsigned long long)dxor);
+    atomicAdd(&w.vars[V_NHITS], (unsigned long long)nh);
+  }
+}
+
+__global__ void k_grep_close(const gfs_ctx* c, GrepWork w) {
+  const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
+  for (uint32_t f = blockIdx.x; f < nfiles; f += gridDim.x) {
+    const int fd = w.fd[f];
+    if (fd >= 0) gclose(c, fd);
+  }
+}
+
+// unique records from the (file, word) table + word totals
+__global__ void k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap, uint64_t* totals) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i <= w.pair_mask; i += stride) {
+    const uint64_t key = w.pair_key[i];
+    if (key == kPairEmpty) continue;
+    const uint64_t cnt = w.pair_cnt[i];
+    const uint32_t k = (uint32_t)key;
+    atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
+    const unsigned long long idx = atomicAdd(&w.vars[V_NREC], 1ull);
+    if (idx < rec_cap) {
+      rec[3 * idx] = (uint32_t)(key >> 32);
+      rec[3 * idx + 1] = k;
+      rec[3 * idx + 2] = (uint32_t)cnt;
+    }
+  }
+}
+
+__global__ void k_grep_init(GrepWork w, uint32_t max_words) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
+  for (uint64_t i = t; i <= w.pair_mask; i += stride) {
+    w.pair_key[i] = kPairEmpty;
+    w.pair_cnt[i] = 0;
+  }
+  for (uint64_t i = t; i <= w.table_mask; i += stride) w.table[i] = 0;
+  for (uint64_t i = t; i < max_words; i += stride) {
+    w.dup_head[i] = 0;
+    w.dup_next[i] = 0;
+  }
+  if (t < V_NVARS) w.vars[t] = 0;
+}
+
+__global__ void k_grep_summary(GrepWork w, uint64_t* out) {
+  if (threadIdx.x == 0) {
+    out[0] = w.vars[V_NREC];
+    out[1] = w.vars[V_NHITS];
+    out[2] = w.vars[V_DSUM];
+    out[3] = w.vars[V_DXOR];
+    out[4] = w.vars[V_NFILES];
+    out[5] = w.vars[V_NWORDS];
+    out[6] = w.vars[V_BYTES];
+    out[7] = w.vars[V_ERR];
+    out[8] = w.vars[V_NLISTED];
+    out[9] = w.vars[V_NITEMS];
+  }
+}
+
+uint64_t pow2_at_least(uint64_t x) {
+  uint64_t p = 1;
+  while (p < x) p <<= 1;
+  return p;
+}
+
+struct Layout {
+  uint64_t off[16];
+  uint64_t total;
+};
+
+Layout layout(const gfs_grep_params* p) {
+  Layout L{};
+  const uint64_t tcap = pow2_at_least(p->max_words * 2ull < 1024 ? 1024 : p->max_words * 2ull);
+  const uint64_t pcap = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap);
+  const uint64_t sizes[] = {
+      (uint64_t)p->max_words * 32,         // dict
+      tcap * 8,                            // table
+      (uint64_t)p->max_words * 4,          // dup_head
+      (uint64_t)p->max_words * 4,          // dup_next
+      p->list_cap + 64,                    // list
+      (uint64_t)p->max_files * kMaxPath,   // paths
+      (uint64_t)p->max_files * 4,          // path_len
+      (uint64_t)p->max_files * 4,          // fd
+      (uint64_t)p->max_files * 8,          // size
+      ((uint64_t)p->max_files + 1) * 8,    // item_base
+      pcap * 8,                            // pair_key
+      pcap * 8,                            // pair_cnt
+      V_NVARS * 8,                         // vars
+  };
+  uint64_t o = 0;
+  for (int i = 0; i < 13; ++i) {
+    L.off[i] = o;
+    o += (sizes[i] + 255) & ~255ull;
+  }
+  L.total = o;
+  return L;
+}
+
+}  // namespace
+
+GFS_API uint64_t gfs_grep_work_bytes(const gfs_grep_params* p) { return p ? layout(p).total : 0; }
+
+GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
+                     const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
+                     uint64_t* d_hits, uint64_t* d_summary) {
+  if (!h || !dict_path || !list_path || !p || !d_work || !d_totals || !d_summary || p->max_files == 0 ||
+      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) || p->grid == 0 ||
+      p->block == 0 || p->block > 256 || (p->block & 31))
+    return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const Layout L = layout(p);
+  uint8_t* base = (uint8_t*)d_work;
+  GrepWork w;
+  w.dict = base + L.off[0];
+  w.table = (uint64_t*)(base + L.off[1]);
+  w.table_mask = (uint32_t)(pow2_at_least(p->max_words * 2ull < 1024 ? 1024 : p->max_words * 2ull) - 1);
+  w.dup_head = (uint32_t*)(base + L.off[2]);
+  w.dup_next = (uint32_t*)(base + L.off[3]);
+  w.list = base + L.off[4];
+  w.paths = (char*)(base + L.off[5]);
+  w.path_len = (uint32_t*)(base + L.off[6]);
+  w.fd = (int32_t*)(base + L.off[7]);
+  w.size = (uint64_t*)(base + L.off[8]);
+  w.item_base = (uint64_t*)(base + L.off[9]);
+  w.pair_key = (uint64_t*)(base + L.off[10]);
+  w.pair_cnt = (uint64_t*)(base + L.off[11]);
+  w.pair_mask = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap) - 1;
+  w.vars = (unsigned long long*)(base + L.off[12]);
+
+  // staged strings: dict path, list path, list directory
+  static char* d_str = nullptr;
+  static char* h_str = nullptr;
+  static cudaEvent_t ev = nullptr;
+  if (!d_str) {
+    if (cudaMalloc((void**)&d_str, 3 * kMaxPath) != cudaSuccess) return -ENOMEM;
+    if (cudaHostAlloc((void**)&h_str, 3 * kMaxPath, cudaHostAllocPortable) != cudaSuccess) return -ENOMEM;
+    cudaEventCreateWithFlags(&ev, cudaEventDisableTiming);
+  } else {
+    cudaEventSynchronize(ev);
+  }
+  const size_t nd = strlen(dict_path), nl = strlen(list_path);
+  if (nd >= kMaxPath || nl >= kMaxPath) return -ENAMETOOLONG;
+  memcpy(h_str, dict_path, nd + 1);
+  memcpy(h_str + kMaxPath, list_path, nl + 1);
+  const char* slash = strrchr(list_path, '/');
+  size_t dl = 0;
+  if (slash) {
+    dl = (size_t)(slash - list_path);
+    memcpy(h_str + 2 * kMaxPath, list_path, dl);
+  } else {
+    h_str[2 * kMaxPath] = '.';
+    dl = 1;
+  }
+  h_str[2 * kMaxPath + dl] = 0;
+  cudaMemcpyAsync(d_str, h_str, 3 * kMaxPath, cudaMemcpyHostToDevice, s);
+  cudaEventRecord(ev, s);
+
+  const gfs_ctx* c = gfs_device_ctx(h);
+  const uint32_t smem = ((p->chunk + kPre + kHalo + 15) & ~15u) + 2 * kCountSlots * 4;
+  if (smem > 227 * 1024) return -EINVAL;
+  cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  // GFS_GREP_DEBUG=1: synchronise after each stage and report the first failing one
+  const bool dbg = getenv("GFS_GREP_DEBUG") && *getenv("GFS_GREP_DEBUG") == '1';
+  auto stage = [&](const char* name) {
+    if (!dbg) return;
+    cudaError_t e = cudaStreamSynchronize(s);
+    long long err = 0;
+    cudaMemcpy(&err, &w.vars[V_ERR], 8, cudaMemcpyDeviceToHost);
+    unsigned long long v[V_NVARS];
+    cudaMemcpy(v, w.vars, sizeof(v), cudaMemcpyDeviceToHost);
+    fprintf(stderr, "gfs_grep[%s]: cuda=%s err=%lld nfiles=%llu nwords=%llu nitems=%llu bytes=%llu\n", name,
+            cudaGetErrorString(e), err, v[V_NFILES], v[V_NWORDS], v[V_NITEMS], v[V_BYTES]);
+  };
+  k_grep_init<<<1024, 256, 0, s>>>(w, p->max_words);
+  const uint32_t dict_blocks = 64;
+  k_grep_dict<<<dict_blocks, 256, 0, s>>>(c, d_str, w, p->max_words);
+  stage("dict");
+  k_grep_list<<<1, 256, 0, s>>>(c, d_str + kMaxPath, d_str + 2 * kMaxPath, (uint32_t)dl, w, p->list_cap,
+                                 p->max_files);
+  stage("list");
+  k_grep_open<<<p->grid, 128, 0, s>>>(c, w, p->chunk);
+  stage("open");
+  k_grep_plan<<<1, 1024, 0, s>>>(w);
+  k_grep_scan<<<p->grid, p->block, smem, s>>>(c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0);
+  stage("scan");
+  if (!p->keep_open) k_grep_close<<<p->grid, 32, 0, s>>>(c, w);
+  cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
+  k_grep_compact<<<1024, 256, 0, s>>>(w, d_rec, d_rec ? rec_cap : 0, d_totals);
+  k_grep_summary<<<1, 32, 0, s>>>(w, d_summary);
+  stage("done");
+  const cudaError_t e = cudaGetLastError();
+  if (e != cudaSuccess) fprintf(stderr, "gfs_grep: launch failed: %s\n", cudaGetErrorString(e));
+  return e == cudaSuccess ? 0 : -EIO;
+}

@@ -7,14 +7,18 @@
 //     memory, one queue per GPU owned by that GPU; a slot is
 //     published by the GPU with st.release.sys on its seq word;
 //   * W worker threads (not the paper's single event thread) each
-//     claim the next ticket, spin on its slot, pread into a pinned staging
-//     buffer (double-buffered per worker) and cudaMemcpyAsync it into the
-//     cache frame on the worker's own non-blocking stream;
-//   * completion is stream-ordered after the DMA: cuStreamWriteValue64 of
-//     ((ticket+1) << 32 | result) into a completion word in HBM, which the
-//     waiting GPU thread polls locally (no PCIe reads on the GPU side);
-//   * dirty ranges come back by D2H + pwrite; a partially written range is
-//     merged with the host copy by "diff against zeros";
+//     claim the next ticket, spin on its slot and serve it with POSIX calls
+//     only: READ preads into the pinned staging slot the GPU named, WRITE
+//     pwrites from it, OPEN/CLOSE/TRUNC act on the fd table;
+//   * completion is a store-release of ((ticket+1) << 32 | result) into a
+//     pinned completion word that the waiting GPU thread polls with
+//     ld.acquire.sys. The daemon makes NO CUDA call per request: a
+//     stream-ordered DMA or stream write-value can be queued behind the very
+//     kernel that waits for it when the streams share a hardware queue
+//     (CUDA_DEVICE_MAX_CONNECTIONS), so the GPU pulls pages out of staging
+//     itself (and pushes dirty ranges into it for write-back);
+//   * a partially written dirty range is merged with the host copy by "diff
+//     against zeros";
 //   * close-to-open consistency uses a shared-memory version table keyed by
 //     (st_dev, st_ino), bumped on every write-back (stand-in for WRAPFS,
 //     P:L760-772); OPEN replies carry it so re-opens can validate.
@@ -34,20 +38,15 @@
 #include <unistd.h>
 #include <vector>
 
-#include <cuda.h>
 #include <cuda_runtime.h>
 
 #include "gpufs.h"
 
 #define GFS_API extern "C" __attribute__((visibility("default")))
 
-// Launchers live in gfs_kernels.cu; they need these.
 extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s);
 
 namespace {
-
-typedef CUresult (*PFN_writeValue64)(CUstream, CUdeviceptr, cuuint64_t, unsigned int);
-typedef CUresult (*PFN_devAttr)(int*, CUdevice_attribute, CUdevice);
 
 inline void cpu_relax() {
 #if defined(__x86_64__)
@@ -158,39 +157,30 @@ struct HostFile {
   uint64_t dev = 0, ino = 0;
 };
 
-struct gfs_handle;
-
 struct Worker {
   std::thread th;
-  cudaStream_t stream = nullptr;
-  uint8_t* staging[2] = {nullptr, nullptr};
-  cudaEvent_t ev[2] = {nullptr, nullptr};
-  bool pending[2] = {false, false};
-  int cur = 0;
   std::vector<uint8_t> merge;
 };
 
 struct gfs_handle {
   gfs_config cfg{};
-  gfs_ctx h{};         // host copy holding device pointers
+  gfs_ctx h{};           // host copy holding device pointers
   gfs_ctx* d = nullptr;  // device copy
   bool own_pool = false;
   cudaStream_t priv = nullptr;
   gfs_rpc_req* ring_h = nullptr;
   gfs_rpc_resp* resp_h = nullptr;
   char* paths_h = nullptr;
-  uint64_t* cplsrc_h = nullptr;
+  uint64_t* cpl_h = nullptr;
+  uint8_t* staging_h = nullptr;
   std::vector<Worker> workers;
   std::atomic<uint64_t> next_ticket{0};
   std::atomic<bool> running{false};
-  std::thread runner_dummy;
   std::mutex fd_mu;
   std::vector<HostFile> files;
   std::vector<uint32_t> free_hfids;
-  PFN_writeValue64 wv64 = nullptr;
   VersionTable vt;
   std::atomic<uint64_t> hs[HS_N];
-  uint64_t staging_bytes = 0;
 };
 
 namespace {
@@ -237,30 +227,12 @@ void free_hfid(gfs_handle* h, uint32_t id) {
   h->free_hfids.push_back(id);
 }
 
-void complete(gfs_handle* h, Worker& w, uint32_t slot, uint64_t ticket, int32_t result) {
-  const uint64_t v = ((ticket + 1) << 32) | (uint32_t)result;
-  CUdeviceptr addr = (CUdeviceptr)(h->h.cpl + slot);
-  if (h->wv64) {
-    CUresult r = h->wv64((CUstream)w.stream, addr, v, 0);
-    if (r == CUDA_SUCCESS) return;
-  }
-  // Fallback: an 8-byte H2D copy from a per-slot pinned source, ordered after the DMA.
-  h->cplsrc_h[slot] = v;
-  cudaMemcpyAsync((void*)addr, &h->cplsrc_h[slot], 8, cudaMemcpyHostToDevice, w.stream);
+inline void complete(gfs_handle* h, uint32_t slot, uint64_t ticket, int32_t result) {
+  __atomic_store_n(&h->cpl_h[slot], ((ticket + 1) << 32) | (uint32_t)result, __ATOMIC_RELEASE);
 }
 
-uint8_t* staging_acquire(Worker& w) {
-  const int b = w.cur;
-  if (w.pending[b]) {
-    cudaEventSynchronize(w.ev[b]);
-    w.pending[b] = false;
-  }
-  return w.staging[b];
-}
-void staging_issued(Worker& w) {
-  cudaEventRecord(w.ev[w.cur], w.stream);
-  w.pending[w.cur] = true;
-  w.cur ^= 1;
+inline uint8_t* staging_slot(gfs_handle* h, uint32_t stage) {
+  return h->staging_h + ((size_t)stage << h->h.page_shift);
 }
 
 int32_t do_open(gfs_handle* h, uint32_t slot, const gfs_rpc_req& q) {
@@ -311,22 +283,17 @@ int32_t do_open(gfs_handle* h, uint32_t slot, const gfs_rpc_req& q) {
   return 0;
 }
 
-int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
+int32_t do_read(gfs_handle* h, const gfs_rpc_req& q) {
   HostFile f = get_hfid(h, q.hfid);
   if (f.fd < 0) return -EBADF;
-  if (q.len > h->staging_bytes) return -EINVAL;
-  uint8_t* buf = staging_acquire(w);
+  if (q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
+  uint8_t* buf = staging_slot(h, q.stage);
   auto t0 = std::chrono::steady_clock::now();
   int64_t n = pread_full(f.fd, buf, q.len, q.file_off);
   h->hs[HS_PREAD_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
                             std::chrono::steady_clock::now() - t0).count();
   if (n < 0) return (int32_t)n;
   if ((uint64_t)n < q.len) memset(buf + n, 0, q.len - (size_t)n);  // host file shrank: zeros (R4)
-  if (q.len) {
-    cudaError_t e = cudaMemcpyAsync((void*)q.dev_ptr, buf, q.len, cudaMemcpyHostToDevice, w.stream);
-    if (e != cudaSuccess) return -EIO;
-    staging_issued(w);
-  }
   h->hs[HS_READ]++;
   h->hs[HS_BYTES_H2D] += q.len;
   return (int32_t)q.len;
@@ -336,13 +303,9 @@ int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   HostFile f = get_hfid(h, q.hfid);
   if (f.fd < 0) return -EBADF;
   if (!(f.mode & GFS_O_GWRONCE)) return -EBADF;  // read-only files are never written back
-  if (q.len > h->staging_bytes) return -EINVAL;
-  uint8_t* buf = staging_acquire(w);
-  if (q.len) {
-    if (cudaMemcpyAsync(buf, (const void*)q.dev_ptr, q.len, cudaMemcpyDeviceToHost, w.stream) != cudaSuccess)
-      return -EIO;
-    if (cudaStreamSynchronize(w.stream) != cudaSuccess) return -EIO;
-  }
+  const uint64_t in_page = q.file_off & (h->h.page_size - 1);
+  if (in_page + q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
+  uint8_t* buf = staging_slot(h, q.stage) + in_page;
   if (!(q.flags & GFS_WF_FULL)) {
     // Not every byte of the range was written: diff against zeros.
     w.merge.assign(q.len, 0);
@@ -361,7 +324,6 @@ int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
 }
 
 void worker_loop(gfs_handle* h, int wi) {
-  cudaSetDevice(h->cfg.device);
   Worker& w = h->workers[wi];
   const uint32_t R = h->h.ring_slots;
   while (h->running.load(std::memory_order_acquire)) {
@@ -394,9 +356,10 @@ void worker_loop(gfs_handle* h, int wi) {
     q.flags = vq->flags;
     q.arg = vq->arg;
     q.path_len = vq->path_len;
+    q.stage = vq->stage;
     int32_t res;
     switch (q.op) {
-      case GFS_OP_READ: res = do_read(h, w, q); break;
+      case GFS_OP_READ: res = do_read(h, q); break;
       case GFS_OP_WRITE: res = do_write(h, w, q); break;
       case GFS_OP_OPEN: res = do_open(h, slot, q); break;
       case GFS_OP_CLOSE:
@@ -416,9 +379,8 @@ void worker_loop(gfs_handle* h, int wi) {
     }
     if (res < 0) h->hs[HS_ERRORS]++;
     h->hs[HS_RPC]++;
-    complete(h, w, slot, t, res);
+    complete(h, slot, t, res);
   }
-  cudaStreamSynchronize(w.stream);
 }
 
 void free_all(gfs_handle* h) {
@@ -429,18 +391,12 @@ void free_all(gfs_handle* h) {
   F(h->h.f_state); F(h->h.f_tag); F(h->h.f_file); F(h->h.f_valid); F(h->h.f_lo); F(h->h.f_hi);
   F(h->h.f_written); F(h->h.f_stamp); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
   F(h->h.node_free); F(h->h.node_free_top); F(h->h.node_lock); F(h->h.files); F(h->h.paths); F(h->h.uid_next);
-  F(h->h.cpl); F(h->h.ack); F(h->h.ring_tail); F(h->h.ctr); F(h->d);
+  F(h->h.ack); F(h->h.ring_tail); F(h->h.ctr); F(h->h.staging_bits); F(h->d);
   if (h->ring_h) cudaFreeHost(h->ring_h);
   if (h->resp_h) cudaFreeHost(h->resp_h);
   if (h->paths_h) cudaFreeHost(h->paths_h);
-  if (h->cplsrc_h) cudaFreeHost(h->cplsrc_h);
-  for (auto& w : h->workers) {
-    for (int b = 0; b < 2; ++b) {
-      if (w.staging[b]) cudaFreeHost(w.staging[b]);
-      if (w.ev[b]) cudaEventDestroy(w.ev[b]);
-    }
-    if (w.stream) cudaStreamDestroy(w.stream);
-  }
+  if (h->cpl_h) cudaFreeHost(h->cpl_h);
+  if (h->staging_h) cudaFreeHost(h->staging_h);
   if (h->priv) cudaStreamDestroy(h->priv);
   for (auto& f : h->files)
     if (f.fd >= 0) ::close(f.fd);
@@ -463,6 +419,7 @@ GFS_API int gfs_config_default(gfs_config* c) {
   c->max_nodes = 0;
   c->max_batch = GFS_MAX_BATCH;
   c->flags = 0;
+  c->staging_slots = 0;
   c->timeout_ms = 60000;
   return 0;
 }
@@ -485,8 +442,14 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   gfs_ctx& c = h->h;
   const uint32_t R = cfg->ring_slots;
   const uint32_t MF = cfg->max_files;
-  uint32_t max_nodes = cfg->max_nodes ? cfg->max_nodes : (MF * 2u + 65536u);
-  size_t ctr_bytes = (size_t)GFS_C_NCOUNTERS * GFS_CTR_SHARDS * sizeof(unsigned long long);
+  const uint32_t max_nodes = cfg->max_nodes ? cfg->max_nodes : (MF * 2u + 65536u);
+  const size_t ctr_bytes = (size_t)GFS_C_NCOUNTERS * GFS_CTR_SHARDS * sizeof(unsigned long long);
+  uint32_t slots = cfg->staging_slots;
+  if (!slots) {
+    const uint64_t want = (128ull << 20) / cfg->page_size;
+    slots = (uint32_t)(want < 32 ? 32 : (want > 4096 ? 4096 : want));
+  }
+  const uint32_t words = (slots + 31) / 32;
 
   CK(cudaSetDevice(cfg->device));
   CK(cudaFree(0));
@@ -524,13 +487,20 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaHostAlloc((void**)&h->ring_h, (size_t)R * sizeof(gfs_rpc_req), cudaHostAllocMapped | cudaHostAllocPortable));
   CK(cudaHostAlloc((void**)&h->resp_h, (size_t)R * sizeof(gfs_rpc_resp), cudaHostAllocMapped | cudaHostAllocPortable));
   CK(cudaHostAlloc((void**)&h->paths_h, (size_t)R * GFS_MAX_PATH, cudaHostAllocMapped | cudaHostAllocPortable));
-  CK(cudaHostAlloc((void**)&h->cplsrc_h, (size_t)R * 8, cudaHostAllocPortable));
+  CK(cudaHostAlloc((void**)&h->cpl_h, (size_t)R * 8, cudaHostAllocMapped | cudaHostAllocPortable));
+  CK(cudaHostAlloc((void**)&h->staging_h, (size_t)slots * cfg->page_size,
+                   cudaHostAllocMapped | cudaHostAllocPortable));
   memset(h->ring_h, 0, (size_t)R * sizeof(gfs_rpc_req));
   memset(h->resp_h, 0, (size_t)R * sizeof(gfs_rpc_resp));
+  memset(h->cpl_h, 0, (size_t)R * 8);
   CK(cudaHostGetDevicePointer((void**)&c.ring, h->ring_h, 0));
   CK(cudaHostGetDevicePointer((void**)&c.resp, h->resp_h, 0));
   CK(cudaHostGetDevicePointer((void**)&c.ring_paths, h->paths_h, 0));
-  CK(cudaMalloc((void**)&c.cpl, (size_t)R * 8));
+  CK(cudaHostGetDevicePointer((void**)&c.cpl, h->cpl_h, 0));
+  CK(cudaHostGetDevicePointer((void**)&c.staging, h->staging_h, 0));
+  c.staging_slots = slots;
+  c.staging_words = words;
+  CK(cudaMalloc((void**)&c.staging_bits, (size_t)words * 4));
   CK(cudaMalloc((void**)&c.ack, (size_t)R * 8));
   CK(cudaMalloc((void**)&c.ring_tail, 8));
   CK(cudaMalloc((void**)&c.ctr, ctr_bytes));
@@ -540,7 +510,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMemsetAsync(c.nodes, 0, (size_t)max_nodes * GFS_FANOUT * 4, h->priv));
   CK(cudaMemsetAsync(c.files, 0, (size_t)MF * sizeof(gfs_file), h->priv));
   CK(cudaMemsetAsync(c.paths, 0, (size_t)MF * GFS_MAX_PATH, h->priv));
-  CK(cudaMemsetAsync(c.cpl, 0, (size_t)R * 8, h->priv));
+  CK(cudaMemsetAsync(c.staging_bits, 0, (size_t)words * 4, h->priv));
   CK(cudaMemsetAsync(c.ack, 0, (size_t)R * 8, h->priv));
   CK(cudaMemsetAsync(c.ring_tail, 0, 8, h->priv));
   CK(cudaMemsetAsync(c.ctr, 0, ctr_bytes, h->priv));
@@ -554,33 +524,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMalloc((void**)&h->d, sizeof(gfs_ctx)));
   CK(cudaMemcpyAsync(h->d, &c, sizeof(gfs_ctx), cudaMemcpyHostToDevice, h->priv));
   CK(cudaStreamSynchronize(h->priv));
-
-  // stream write-value-64 for completions (CUDA 12: attribute 122)
-  {
-    void* fn = nullptr;
-    cudaDriverEntryPointQueryResult q;
-    if (!(cfg->flags & GFS_F_NO_DMA_COMPLETION) &&
-        cudaGetDriverEntryPoint("cuStreamWriteValue64", &fn, cudaEnableDefault, &q) == cudaSuccess &&
-        q == cudaDriverEntryPointSuccess && fn) {
-      void* fa = nullptr;
-      int ok = 0;
-      if (cudaGetDriverEntryPoint("cuDeviceGetAttribute", &fa, cudaEnableDefault, &q) == cudaSuccess && fa) {
-        CUdevice dev = cfg->device;
-        ((PFN_devAttr)fa)(&ok, (CUdevice_attribute)122 /* CAN_USE_64_BIT_STREAM_MEM_OPS */, dev);
-      }
-      if (ok) h->wv64 = (PFN_writeValue64)fn;
-    }
-  }
-
-  h->staging_bytes = cfg->page_size;
   h->workers.resize(cfg->daemon_threads);
-  for (auto& w : h->workers) {
-    CK(cudaStreamCreateWithFlags(&w.stream, cudaStreamNonBlocking));
-    for (int b = 0; b < 2; ++b) {
-      CK(cudaHostAlloc((void**)&w.staging[b], h->staging_bytes, cudaHostAllocPortable));
-      CK(cudaEventCreateWithFlags(&w.ev[b], cudaEventDisableTiming));
-    }
-  }
   if (!h->vt.open()) fprintf(stderr, "gpufs: version table unavailable; close-to-open checks use size/mtime only\n");
   *out = h;
   return 0;
@@ -606,8 +550,8 @@ GFS_API int gfs_daemon_stop(gfs_handle* h) {
   h->running.store(false);
   for (auto& w : h->workers)
     if (w.th.joinable()) w.th.join();
-  // tickets claimed by idle workers are handed out again on restart
-  // (the GPU's tail never passed them); resynchronise with the device tail.
+  // Tickets claimed by idle workers were never posted by the GPU: restart
+  // from the device's tail.
   unsigned long long tail = 0;
   cudaMemcpyAsync(&tail, h->h.ring_tail, 8, cudaMemcpyDeviceToHost, h->priv);
   cudaStreamSynchronize(h->priv);
@@ -658,7 +602,7 @@ GFS_API int gfs_info(gfs_handle* h, uint64_t* out, int n) {
   cudaMemcpyAsync(&tail, h->h.ring_tail, 8, cudaMemcpyDeviceToHost, h->priv);
   cudaStreamSynchronize(h->priv);
   uint64_t v[9] = {h->h.page_size, h->h.nframes, h->h.max_files, h->h.max_nodes, h->h.ring_slots,
-                   h->workers.size(), h->wv64 ? 1u : 0u, h->next_ticket.load(), tail};
+                   h->workers.size(), h->h.staging_slots, h->next_ticket.load(), tail};
   for (int i = 0; i < n && i < 9; ++i) out[i] = v[i];
   return 9;
 }

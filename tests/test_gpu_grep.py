@@ -1,0 +1,94 @@
+"""GPU parity for the grep -w consumer (C1, C4 shapes) vs the oracle: bit-exact
+records, totals, hit digest and (C1 / small cases) the full hit list."""
+import json
+import os
+
+import numpy as np
+import pytest
+
+import gen
+import oracle
+
+pytestmark = [pytest.mark.gpu, pytest.mark.timeout(900)]
+GOLD = os.path.join(os.path.dirname(__file__), "golden")
+
+
+@pytest.fixture(scope="module")
+def g():
+    import paper_conf_asplos_silbersteinfkw13_b200 as g
+    g.build.build()
+    return g
+
+
+def compare(got, ref, hits=True):
+    assert got["summary"]["err"] == 0, got["summary"]
+    assert got["summary"]["nfiles"] == ref.nfiles
+    assert got["summary"]["bytes"] == ref.bytes
+    assert got["records"].tolist() == ref.records.tolist()
+    assert got["totals"].tolist() == ref.totals.tolist()
+    assert got["digest"] == ref.digest
+    if hits:
+        assert got["hits"].tolist() == ref.hits.tolist()
+
+
+@pytest.mark.parametrize("chunk,P", [(16, 4096), (48, 4096), (4096, 4096), (32768, 65536)])
+def test_hand_golden(g, shmdir, chunk, P):
+    d = json.load(open(os.path.join(GOLD, "grep_hand.json")))
+    paths = []
+    for i, hx in enumerate(d["files_hex"]):
+        p = os.path.join(shmdir, f"h{i}.txt")
+        open(p, "wb").write(bytes.fromhex(hx))
+        paths.append(p)
+    gen.write_dict(os.path.join(shmdir, "d.bin"), [w.encode() for w in d["words"]])
+    gen.write_list(os.path.join(shmdir, "l.txt"), paths)
+    with g.GpuFS(cache_bytes=64 * P, page_size=P, timeout_ms=30000, daemon_threads=2) as fs:
+        out = fs.grep(os.path.join(shmdir, "d.bin"), os.path.join(shmdir, "l.txt"), hits=True, chunk=chunk, grid=8)
+    assert out["summary"]["err"] == 0
+    assert out["records"].tolist() == d["expected_records"]
+    assert out["totals"].tolist() == d["expected_totals"]
+    assert out["hits"].tolist() == d["expected_hits"]
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_tiny_random_vs_oracle(g, shmdir, seed):
+    extra = [b"", b"ab", b"b" * 32 + b" " + b"b" * 33, b"a" * 40, b"ab " * 2000]
+    c = gen.tiny_corpus(shmdir, seed, nfiles=6, max_bytes=5000, nwords=10, extra_files=extra,
+                        extra_words=[b"b" * 32, b"ab", b"ab"])
+    ref = oracle.grep_brute(c["dict"], c["list"])
+    chunk = [16, 32, 64, 128, 1024, 4096][seed]
+    with g.GpuFS(cache_bytes=32 * 4096, page_size=4096, timeout_ms=30000, daemon_threads=2, max_batch=2) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=True, chunk=chunk, grid=16)
+    compare(out, ref)
+
+
+def test_c1_vs_oracle(g, shmdir):
+    c = gen.c1_corpus(os.path.join(shmdir, "c1"), seed=1)
+    ref = oracle.grep(c["dict"], c["list"], nthreads=4)
+    with g.GpuFS(cache_bytes=1 << 30, page_size=64 << 10, timeout_ms=30000, daemon_threads=4) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=True)
+        out2 = fs.grep(c["dict"], c["list"], hits=True)  # warm: cache reused across launches
+        st = fs.stats()
+    compare(out, ref)
+    compare(out2, ref)
+    assert st["reopen_valid"] > 0
+
+
+def test_c4_shape_small_vs_oracle(g, shmdir):
+    c = gen.c4_corpus(os.path.join(shmdir, "c4"), seed=4, nfiles=1500, total_bytes=24 << 20, nwords=58000)
+    ref = oracle.grep(c["dict"], c["list"], want_hits=False, nthreads=8)
+    with g.GpuFS(cache_bytes=1 << 30, page_size=64 << 10, timeout_ms=60000, daemon_threads=8,
+                 max_files=4096) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=False)
+    compare(out, ref, hits=False)
+    assert out["summary"]["nhits"] == ref.digest[2]
+
+
+def test_cache_smaller_than_corpus(g, shmdir):
+    """Eviction during grep: a 2 MiB cache under an 8 MiB corpus."""
+    c = gen.c1_corpus(os.path.join(shmdir, "c1s"), seed=3, nfiles=8, file_bytes=1 << 20)
+    ref = oracle.grep(c["dict"], c["list"], nthreads=4)
+    with g.GpuFS(cache_bytes=2 << 20, page_size=64 << 10, timeout_ms=60000, daemon_threads=4, max_batch=1) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=True, grid=8)
+        st = fs.stats()
+    compare(out, ref)
+    assert st["evict"] > 0

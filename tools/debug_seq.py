@@ -34,6 +34,6 @@ for case in cases:
     print(f"file={fm}MiB cache={cm}MiB P={pk}K grid={grid} W={w}: err={err} ok={ok} {dt:.2f}s "
           f"{sweeps*size/dt/1e9:.2f} GB/s x{sweeps} | miss={st['miss']} evict={st['evict']} rpc={st['rpc']} timeout={st['timeout']} "
           f"enomem={st['enomem']} ringwait={st['ring_wait']} | host rpc={hs['rpc']} read={hs['read']} err={hs['errors']} "
-          f"pread={hs['bytes_h2d']/max(hs['pread_ns'],1):.2f}GB/s/thr | next={info['host_next_ticket']} tail={info['device_ring_tail']} wv64={info['stream_write_value64']}",
+          f"pread={hs['bytes_h2d']/max(hs['pread_ns'],1):.2f}GB/s/thr | next={info['host_next_ticket']} tail={info['device_ring_tail']} stage={info['staging_slots']} busy={st['busy']}",
           flush=True)
     fs.close()
