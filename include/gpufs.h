@@ -155,6 +155,7 @@ typedef struct gfs_grep_params {
   uint32_t grid;        /* persistent blocks */
   uint32_t block;       /* threads per block, multiple of 32, <= 256 */
   uint32_t keep_open;   /* 1: leave every file open after the run (warm re-runs skip the host) */
+  uint64_t corpus_cap;  /* bytes of all listed files (capacity, sizes the work-item map) */
 } gfs_grep_params;
 
 /* Device scratch bytes gfs_grep needs for these parameters. */

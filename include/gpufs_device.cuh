@@ -286,9 +286,15 @@ __device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64
   q->arg = arg;
   q->path_len = path_len;
   q->stage = (uint32_t)stage;
-  if (path) {
+  if (path) {  // 8-byte stores where aligned: each store is one PCIe write
     volatile char* dp = c->ring_paths + (size_t)slot * GFS_MAX_PATH;
-    for (uint32_t i = 0; i < path_len; ++i) dp[i] = path[i];
+    uint32_t i = 0;
+    if (((uintptr_t)path & 7) == 0) {
+      volatile uint64_t* d8 = (volatile uint64_t*)dp;
+      const uint64_t* s8 = (const uint64_t*)path;
+      for (; i + 8 <= path_len; i += 8) d8[i >> 3] = s8[i >> 3];
+    }
+    for (; i < path_len; ++i) dp[i] = path[i];
   }
   st_rel_sys64((uint64_t*)&q->seq, (uint64_t)(t + 1));
   ctr(c, GFS_C_RPC);
@@ -312,6 +318,7 @@ __device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64
     resp_out->mtime_ns = r->mtime_ns;
     resp_out->hfid = r->hfid;
     resp_out->status = r->status;
+    resp_out->pad[0] = r->pad[0];  // OPEN: bytes of page 0 prefetched into the staging slot
   }
   st_rel64(&c->ack[slot], (uint64_t)(t + 1));
   return res;
@@ -325,19 +332,23 @@ __device__ __forceinline__ void spin_lock(uint32_t* l) {
 __device__ __forceinline__ void spin_unlock(uint32_t* l) { st_rel(l, 0u); }
 
 // Returns a zeroed node index (>= 1; node 0 is reserved as "null"), or 0.
+// Never-used nodes come from a lock-free bump counter (every first gopen
+// needs a root: a source tree opens tens of thousands of files at once);
+// recycled nodes from a locked stack.
 __device__ uint32_t node_alloc(const gfs_ctx* c) {
+  if (ld_rlx(c->node_next) < c->max_nodes) {
+    const uint32_t n = atomicAdd(c->node_next, 1u);
+    if (n < c->max_nodes) {
+      ctr(c, GFS_C_NODES);
+      return n;
+    }
+  }
   uint32_t n = 0;
   spin_lock(c->node_lock);
   uint32_t top = *(volatile uint32_t*)c->node_free_top;
   if (top > 0) {
     n = c->node_free[top - 1];
     *(volatile uint32_t*)c->node_free_top = top - 1;
-  } else {
-    uint32_t nx = *(volatile uint32_t*)c->node_next;
-    if (nx < c->max_nodes) {
-      n = nx;
-      *(volatile uint32_t*)c->node_next = nx + 1;
-    }
   }
   spin_unlock(c->node_lock);
   if (n) ctr(c, GFS_C_NODES);
@@ -689,25 +700,29 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
   Lk out{kBusy, -1, 0, 0};
   const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)page;
   uint32_t* lockp = &c->files[fs.fdx].lock;
-  bool locked = false;
-  if (c->flags & GFS_F_LOCKED_TRAVERSAL) {
-    spin_lock(lockp);
-    locked = true;
-  }
-  int err = 0;
-  uint32_t* slot = walk(c, fs.root, fs.height, page, true, &err);
-  if (!slot) {
-    if (locked) spin_unlock(lockp);
-    out.frame = err ? err : -ENOMEM;
-    return out;
-  }
+  const bool always_lock = (c->flags & GFS_F_LOCKED_TRAVERSAL) != 0;  // K5 ablation
+  bool used_lock = false;
   int attempt = 0;
+  uint32_t* slot = nullptr;
   for (;;) {
-    if (!locked && attempt >= 2) {
+    // The lock (when taken) covers the traversal only: walk, slot read,
+    // reference + validation. Fills and RPCs run unlocked.
+    const bool lk = always_lock || attempt >= 2;
+    if (lk) {
       spin_lock(lockp);
-      locked = true;
+      used_lock = true;
+    }
+    if (!slot) {
+      int err = 0;
+      slot = walk(c, fs.root, fs.height, page, true, &err);
+      if (!slot) {
+        if (lk) spin_unlock(lockp);
+        out.frame = err ? err : -ENOMEM;
+        break;
+      }
     }
     const uint32_t s = ld_acq(slot);
+    bool done = false;
     if (s) {
       const uint32_t f = s - 1;
       const uint32_t old = atom_add_acq(&c->f_state[f], 1u);
@@ -716,21 +731,26 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
         if (!(old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
           ctr(c, GFS_C_HIT);
           out.frame = (int)f;
-          break;
+          done = true;
+        } else {
+          atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+          if (old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
+            ctr(c, GFS_C_BUSY);
+            out.frame = kBusy;
+            done = true;
+          }
+          // ERROR with no fill in flight: stale, install over it
         }
-        atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
-        if (old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
-          ctr(c, GFS_C_BUSY);
-          out.frame = kBusy;
-          break;
-        }
-        // ERROR with no fill in flight: stale, install over it
       } else {
         atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
       }
-      ++attempt;
-      ctr(c, GFS_C_RETRY);
+      if (!done) {
+        ++attempt;
+        ctr(c, GFS_C_RETRY);
+      }
     }
+    if (lk) spin_unlock(lockp);
+    if (done) break;
     // miss (or stale slot): install a new frame for `want`
     const int g = alloc_frame(c, want, fs.fdx);
     if (g < 0) {
@@ -772,8 +792,7 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     ctr(c, GFS_C_BYTES_H2D, nb);
     break;
   }
-  if (locked) {
-    spin_unlock(lockp);
+  if (used_lock) {
     ctr(c, GFS_C_LOCKED);
   } else if (out.frame >= 0) {
     ctr(c, GFS_C_LOCKFREE);
@@ -977,9 +996,9 @@ __device__ __forceinline__ bool same_path(const gfs_ctx* c, const gfs_file* e, u
 
 // Open RPC + install of a fresh incarnation. `e` is held in OPENING/REOPENING.
 __device__ int open_rpc_fill(const gfs_ctx* c, gfs_file* e, uint32_t fdx, uint32_t flags, uint32_t old_hfid_plus1,
-                             gfs_rpc_resp* rs) {
+                             gfs_rpc_resp* rs, int stage = -1) {
   const char* sp = c->paths + (size_t)fdx * GFS_MAX_PATH;
-  const int32_t r = rpc_call(c, GFS_OP_OPEN, 0, 0, -1, 0, flags, old_hfid_plus1, sp, e->path_len, rs);
+  const int32_t r = rpc_call(c, GFS_OP_OPEN, 0, 0, stage, 0, flags, old_hfid_plus1, sp, e->path_len, rs);
   ctr(c, GFS_C_RPC_OPEN);
   if (r < 0) return r;
   if (rs->status < 0) return rs->status;
@@ -1010,8 +1029,20 @@ __device__ __forceinline__ void sr_shift(gfs_file* e, uint32_t from, uint32_t to
   atom_add_rel(&e->sr, (uint32_t)(((to - from) << 24) + (uint32_t)dref));
 }
 
+// Page 0 fetched with the OPEN reply (GFS_O_PREFETCH): installed FILLING|1,
+// the calling block pulls it from `stage` and publishes it.
+struct Prefetch {
+  int frame;
+  int stage;
+  uint32_t nbytes;
+};
+
 // gopen body, run by one thread.
-__device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
+__device__ int open_leader(const gfs_ctx* c, const char* path, int flags_in, Prefetch* pf) {
+  pf->frame = -1;
+  pf->stage = -1;
+  const bool want_pf = (flags_in & (int)GFS_O_PREFETCH) != 0;
+  const int flags = flags_in & ~(int)GFS_O_PREFETCH;
   if (flags != (int)GFS_O_RDONLY && flags != (int)GFS_O_GWRONCE) return -EINVAL;
   uint32_t n = 0;
   while (n < GFS_MAX_PATH && path[n]) ++n;
@@ -1041,12 +1072,35 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags) {
       // below): every state change is an atomic delta, never a plain store.
       sr_shift(e, GFS_FS_CLAIM, GFS_FS_OPENING, 0);
       gfs_rpc_resp rs;
-      int r = open_rpc_fill(c, e, i, (uint32_t)flags, 0, &rs);
+      const int pst = (want_pf && flags == (int)GFS_O_RDONLY) ? stage_alloc(c) : -1;
+      int r = open_rpc_fill(c, e, i, (uint32_t)flags, 0, &rs, pst);
       if (r == 0) r = new_incarnation(c, e, (uint32_t)flags, rs);
       if (r < 0) {
+        if (pst >= 0) stage_free(c, pst);
         e->err = r;
         sr_shift(e, GFS_FS_OPENING, GFS_FS_DEAD, -1);  // tombstone; a later gopen retries further along
         return r;
+      }
+      if (pst >= 0) {  // install page 0 while nobody else can see the file
+        int ok = 0;
+        const uint32_t nb = (uint32_t)rs.pad[0];
+        uint32_t* slot = nb ? walk(c, e->root, e->height, 0, true, nullptr) : nullptr;
+        if (slot) {
+          const int g = alloc_frame(c, (uint64_t)e->uid << 32, i);
+          if (g >= 0) {
+            if (atom_cas(slot, 0u, (uint32_t)g + 1u) == 0u) {
+              pf->frame = g;
+              pf->stage = pst;
+              pf->nbytes = nb;
+              ok = 1;
+              ctr(c, GFS_C_MISS);
+              ctr(c, GFS_C_BYTES_H2D, nb);
+            } else {
+              frame_abandon(c, (uint32_t)g);
+            }
+          }
+        }
+        if (!ok) stage_free(c, pst);
       }
       sr_shift(e, GFS_FS_OPENING, GFS_FS_OPEN, 0);
       return (int)i;
@@ -1153,12 +1207,20 @@ __device__ int close_leader(const gfs_ctx* c, int fd) {
 using detail::Scratch;
 
 // gopen: returns an fd shared by all openers of the path on this GPU.
+// flags: GFS_O_RDONLY or GFS_O_GWRONCE, optionally | GFS_O_PREFETCH (hint:
+// when the open goes to the host, page 0 comes back with the reply and the
+// calling block installs it — one RPC instead of two for small files).
 __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
   Scratch& sc = detail::scratch();
+  const int tid = detail::block_tid();
   __syncthreads();
-  if (detail::block_tid() == 0) {
-    const int fd = detail::open_leader(c, path, flags);
+  if (tid == 0) {
+    detail::Prefetch pf;
+    const int fd = detail::open_leader(c, path, flags, &pf);
     sc.ret = fd;
+    sc.frame[0] = pf.frame;
+    sc.stage[0] = pf.stage;
+    sc.nbytes[0] = pf.nbytes;
     sc.cached_fd = -1;
     if (fd >= 0 && detail::snap_fd(c, fd, &sc.cached) && !(sc.cached.oflags & GFS_O_GWRONCE)) {
       sc.cached_grid = detail::grid_id();
@@ -1167,6 +1229,21 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
     }
   }
   __syncthreads();
+  if (sc.frame[0] >= 0) {  // pull the prefetched page 0 and publish it
+    const uint32_t f = (uint32_t)sc.frame[0];
+    detail::block_copy_from_frame<true>(detail::frame_ptr(c, f), detail::stage_ptr(c, sc.stage[0]), sc.nbytes[0],
+                                        tid, detail::block_nthr());
+    __threadfence();
+    __syncthreads();
+    if (tid == 0) {
+      detail::stage_free(c, sc.stage[0]);
+      detail::st_rlx(&c->f_valid[f], sc.nbytes[0]);
+      detail::atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+      detail::frame_release(c, f);
+      sc.frame[0] = -1;
+    }
+    __syncthreads();
+  }
   return (int)sc.ret;
 }
 

@@ -29,6 +29,7 @@ extern "C" {
 /* ---- open flags ------------------------------------------ */
 #define GFS_O_RDONLY 0u
 #define GFS_O_GWRONCE 1u       /* write-once, pages never fetched, pristine = zeros */
+#define GFS_O_PREFETCH 0x100u  /* gopen hint: fetch page 0 with the OPEN reply */
 
 /* ---- config flags ------------------------------------------------------ */
 #define GFS_F_LOCKED_TRAVERSAL 1u /* K5 ablation: every lookup takes the file lock */

@@ -20,7 +20,7 @@ COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", 
             "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
             "ring_wait", "busy", "stage_wait"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
-                 "errors", "merges"]
+                 "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns"]
 
 O_RDONLY = 0
 O_GWRONCE = 1
@@ -45,7 +45,8 @@ class gfs_config(ctypes.Structure):
 class gfs_grep_params(ctypes.Structure):
     _fields_ = [("max_files", ctypes.c_uint32), ("max_words", ctypes.c_uint32), ("list_cap", ctypes.c_uint64),
                 ("pair_cap", ctypes.c_uint64), ("hit_cap", ctypes.c_uint64), ("chunk", ctypes.c_uint32),
-                ("grid", ctypes.c_uint32), ("block", ctypes.c_uint32), ("keep_open", ctypes.c_uint32)]
+                ("grid", ctypes.c_uint32), ("block", ctypes.c_uint32), ("keep_open", ctypes.c_uint32),
+                ("corpus_cap", ctypes.c_uint64)]
 
 
 GREP_SUMMARY = ["nrecords", "nhits", "digest_sum", "digest_xor", "nfiles", "nwords", "bytes", "err",

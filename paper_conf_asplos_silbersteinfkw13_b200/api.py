@@ -173,8 +173,8 @@ class GpuFS:
         return int(d_ret.item())
 
     # grep -w ------------------------------------------------------------------
-    def grep(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
-             pair_cap=1 << 22, hit_cap=None, stream=None, sync=True, state=None):
+    def grep(self, dict_path, list_path, hits=False, chunk=16384, grid=None, block=256, keep_open=False,
+             pair_cap=1 << 22, hit_cap=None, stream=None, sync=True, state=None, corpus_cap=1 << 34):
         """grep -w. Returns a dict with records (n,3) sorted by (file, word),
         totals, digest (sum, xor, nhits), hits (n,3) sorted by (file, offset, word) if requested.
 
@@ -188,8 +188,8 @@ class GpuFS:
             nwords = max(1, os.path.getsize(dict_path) // 32)
             lbytes = os.path.getsize(list_path)
             p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
-                                pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 2 * 148, block=block,
-                                keep_open=1 if keep_open else 0)
+                                pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 4 * 148, block=block,
+                                keep_open=1 if keep_open else 0, corpus_cap=corpus_cap)
             if hits:
                 p.hit_cap = hit_cap if hit_cap is not None else 1 << 22
             work = torch.empty(gfs_grep_work_bytes(p), dtype=torch.uint8, device=dev)
@@ -207,9 +207,9 @@ class GpuFS:
             return state
         s.synchronize()
         summ = dict(zip(GREP_SUMMARY, (int(x) for x in state["summary"].cpu().numpy())))
-        if summ["err"] == -28 and pair_cap < (1 << 30):  # -ENOSPC: (file, word) table too small
+        if summ["err"] == -28 and pair_cap < (1 << 30):  # -ENOSPC: a table was too small
             return self.grep(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap * 4, hit_cap,
-                             stream, sync)
+                             stream, sync, None, corpus_cap * 4)
         out = {"summary": summ}
         nrec = min(summ["nrecords"], p.pair_cap)
         r = state["rec"][:3 * nrec].view(nrec, 3).cpu().numpy().astype(np.uint64)

@@ -9,25 +9,29 @@
 // The paper assigns one dictionary word per thread and brute-forces every
 // position. Here the result is the same (pinned
 // against the brute-force oracle) but the work is proportional to the corpus:
-//   k_grep_dict  gread the dictionary, validate slots, build an open-addressing
-//                hash table (L2-resident) keyed by a 64-bit token hash;
-//   k_grep_list  gread the file list and split it into absolute paths;
-//   k_grep_open  gopen every file once (first gopen goes to the host,
-//                P:L370-372), record fd and size, cut files into work items;
-//   k_grep_plan  exclusive scan of per-file item counts;
-//   k_grep_scan  persistent blocks pull items (file, chunk): gread the chunk
-//                plus a halo into shared memory, find token starts
-//                (W(t[i]) and not W(t[i-1])), hash + probe each token of
-//                <= 32 bytes, count matches per item in shared memory, flush
-//                (file, word) counts into a global table and word totals;
-//   k_grep_close gclose every file (unless kept open for warm re-runs);
-//   k_grep_compact  emit unique (file, word, count) records.
+//   k_grep_dict   gread the dictionary, validate slots, build an open-addressing
+//                 hash table (L2-resident) keyed by a 64-bit token hash;
+//   k_grep_list_* gread the file list in chunks, count line starts per chunk,
+//                 scan, emit absolute paths (parallel over the list);
+//   k_grep_open   gopen every file once (first gopen goes to the host,
+//                 P:L370-372), record fd and size;
+//   k_grep_plan   exclusive scan of per-file work-item counts, item -> file map;
+//   k_grep_scan   persistent blocks pull items (file, chunk): gread the chunk
+//                 plus a halo into shared memory; pass 1 compacts token starts
+//                 (W(t[i]) and not W(t[i-1])) into a shared list, pass 2 gives
+//                 every thread whole tokens (no divergence between lanes): hash +
+//                 probe tokens of <= 32 bytes, count matches per item in shared
+//                 memory, flush (file, word) counts into a global table;
+//   k_grep_close  gclose every file (unless kept open for warm re-runs);
+//   k_grep_compact emit unique (file, word, count) records and word totals.
 // Word bytes are [A-Za-z0-9_] (GNU grep -w under LC_ALL=C, R10).
 #include <cuda_runtime.h>
 #include <errno.h>
 #include <stdint.h>
 #include <stdio.h>
+#include <stdlib.h>
 #include <string.h>
+#include <time.h>
 
 #include "gpufs.h"
 #include "gpufs_device.cuh"
@@ -42,22 +46,26 @@ constexpr uint32_t kMaxPath = GFS_MAX_PATH;
 constexpr uint32_t kHalo = 48;      // bytes after the chunk: a token starting inside may run 33 bytes
 constexpr uint32_t kPre = 16;       // bytes before the chunk (one needed for the boundary test)
 constexpr uint32_t kCountSlots = 2048;
+constexpr uint32_t kListChunk = 65536;
 constexpr uint64_t kPairEmpty = ~0ull;
+constexpr uint64_t kDupBit = 1ull << 63;  // table entry: the word has duplicates
 
 struct GrepWork {
   // dictionary
   uint8_t* dict;          // max_words * 32
-  uint64_t* table;        // dict hash table: (fp32 << 32) | (len << 26) | (k + 1); 0 = empty
+  uint64_t* table;        // (dup << 63) | (fp31 << 32) | (len << 26) | (k + 1); 0 = empty
   uint32_t table_mask;
   uint32_t* dup_head;     // per primary word: first duplicate + 1
   uint32_t* dup_next;     // per word: next duplicate + 1
   // file list
   uint8_t* list;          // list_cap bytes
+  uint32_t* list_chunk;   // per list chunk: line starts (then exclusive prefix)
   char* paths;            // max_files * kMaxPath
-  uint32_t* path_len;
   int32_t* fd;
   uint64_t* size;
   uint64_t* item_base;    // max_files + 1
+  uint32_t* item_file;    // item -> file
+  uint64_t max_items;
   // (file, word) -> count table
   uint64_t* pair_key;
   uint64_t* pair_cnt;
@@ -66,7 +74,7 @@ struct GrepWork {
   unsigned long long* vars;  // see V_*
 };
 enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS, V_DSUM, V_DXOR, V_NLISTED,
-       V_NEXTF, V_NVARS };
+       V_NEXTF, V_LISTSZ, V_NVARS };
 
 __device__ __forceinline__ bool is_word(uint32_t ch) {
   return (ch - 'a' < 26u) || (ch - 'A' < 26u) || (ch - '0' < 10u) || ch == '_';
@@ -79,6 +87,12 @@ __device__ __forceinline__ uint64_t tok_hash(const uint8_t* p, uint32_t n) {
   h *= 0xbf58476d1ce4e5b9ull;
   return h ^ (h >> 32);
 }
+
+// entry bits 32..62 hold a 31-bit fingerprint, 26..31 the length
+__device__ __forceinline__ uint64_t entry_key(uint64_t h, uint32_t len) {
+  return (((h >> 33) & 0x7FFFFFFFull) << 32) | ((uint64_t)len << 26);
+}
+__device__ __forceinline__ uint64_t key_bits(uint64_t e) { return (e & ~kDupBit) >> 26; }
 
 __device__ __forceinline__ uint64_t splitmix64(uint64_t x) {
   uint64_t z = x + 0x9E3779B97F4A7C15ull;
@@ -130,18 +144,19 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
           continue;
         }
         const uint64_t h = tok_hash(s, n);
-        const uint64_t ent = ((h >> 32) << 32) | ((uint64_t)n << 26) | (k + 1);
+        const uint64_t ent = entry_key(h, n) | (k + 1);
         uint32_t slot = (uint32_t)h & w.table_mask;
         for (uint32_t probe = 0; probe <= w.table_mask; ++probe, slot = (slot + 1) & w.table_mask) {
           unsigned long long cur = atomicCAS((unsigned long long*)&w.table[slot], 0ull, (unsigned long long)ent);
           if (cur == 0) break;
-          if ((cur >> 26) == (ent >> 26)) {  // same fingerprint and length: same word?
+          if (key_bits(cur) == key_bits(ent)) {  // same fingerprint and length: same word?
             const uint32_t kp = (uint32_t)(cur & ((1u << 26) - 1)) - 1;
             const uint8_t* t = w.dict + (size_t)kp * 32;
             bool same = true;
             for (uint32_t i = 0; i < n; ++i) same &= t[i] == s[i];
-            if (same) {  // duplicate dictionary word: chain it behind kp
+            if (same) {  // duplicate dictionary word: chain it behind kp, flag the entry
               w.dup_next[k] = atomicExch(&w.dup_head[kp], k + 1);
+              atomicOr((unsigned long long*)&w.table[slot], (unsigned long long)kDupBit);
               break;
             }
           }
@@ -153,52 +168,92 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
 }
 
 // --------------------------------------------------------------- file list
-// One block: read the list, find non-empty lines, emit absolute paths.
-__global__ void k_grep_list(const gfs_ctx* c, const char* list_path, const char* dir, uint32_t dir_len,
-                            GrepWork w, uint64_t list_cap, uint32_t max_files) {
-  __shared__ uint32_t warp_tot[32];
-  __shared__ uint32_t base_s;
-  const int tid = threadIdx.x, nthr = blockDim.x;
+// Pass 1: every block greads its 64 KiB chunks of the list file.
+__global__ void k_grep_list_read(const gfs_ctx* c, const char* list_path, GrepWork w, uint64_t list_cap) {
   const int fd = gopen(c, list_path, GFS_O_RDONLY);
   if (fd < 0) {
-    if (tid == 0) set_err(w, fd);
+    if (threadIdx.x == 0 && blockIdx.x == 0) set_err(w, fd);
     return;
   }
   const int64_t size = gfstat_size(c, fd);
   if (size > (int64_t)list_cap) {
-    if (tid == 0) set_err(w, -ENOSPC);
-    gclose(c, fd);
-    return;
+    if (threadIdx.x == 0 && blockIdx.x == 0) set_err(w, -ENOSPC);
+  } else {
+    if (threadIdx.x == 0 && blockIdx.x == 0) w.vars[V_LISTSZ] = (unsigned long long)size;
+    for (uint64_t o = (uint64_t)blockIdx.x * kListChunk; o < (uint64_t)size; o += (uint64_t)gridDim.x * kListChunk) {
+      const uint64_t n = min((uint64_t)kListChunk, (uint64_t)size - o);
+      const int64_t r = gread(c, fd, o, n, w.list + o);
+      if (r != (int64_t)n && threadIdx.x == 0) set_err(w, r < 0 ? r : -EIO);
+    }
   }
-  const int64_t r = gread(c, fd, 0, (uint64_t)size, w.list);
   gclose(c, fd);
-  if (r != size) {
-    if (tid == 0) set_err(w, r < 0 ? r : -EIO);
-    return;
-  }
-  if (tid == 0) base_s = 0;
-  __syncthreads();
-  const uint8_t* L = w.list;
-  // tiles of nthr bytes: thread i checks byte (tile + i) for a line start
-  for (int64_t t0 = 0; t0 < size; t0 += nthr) {
-    const int64_t i = t0 + tid;
-    bool start = false;
-    if (i < size) start = L[i] != '\n' && (i == 0 || L[i - 1] == '\n');
-    const uint32_t bal = __ballot_sync(0xFFFFFFFFu, start);
-    const int lane = tid & 31, wid = tid >> 5;
-    if (lane == 0) warp_tot[wid] = __popc(bal);
+}
+
+__device__ __forceinline__ bool line_start(const uint8_t* L, uint64_t i) {
+  return L[i] != '\n' && (i == 0 || L[i - 1] == '\n');
+}
+
+// Pass 2: line starts (non-empty lines) per chunk.
+__global__ void k_grep_list_count(GrepWork w) {
+  __shared__ uint32_t cnt_s;
+  const uint64_t size = w.vars[V_LISTSZ];
+  const uint64_t nch = (size + kListChunk - 1) / kListChunk;
+  for (uint64_t ch = blockIdx.x; ch < nch; ch += gridDim.x) {
+    if (threadIdx.x == 0) cnt_s = 0;
     __syncthreads();
-    uint32_t before = base_s;
-    for (int q = 0; q < wid; ++q) before += warp_tot[q];
-    before += __popc(bal & ((1u << lane) - 1));
-    if (start) {
-      const uint32_t k = before;
-      if (k < max_files) {
+    const uint64_t a = ch * kListChunk, b = min(size, a + kListChunk);
+    uint32_t n = 0;
+    for (uint64_t i = a + threadIdx.x; i < b; i += blockDim.x) n += line_start(w.list, i);
+    atomicAdd(&cnt_s, n);
+    __syncthreads();
+    if (threadIdx.x == 0) w.list_chunk[ch] = cnt_s;
+    __syncthreads();
+  }
+}
+
+// Pass 3 (one block): exclusive scan of the chunk counts.
+__global__ void k_grep_list_scan(GrepWork w, uint32_t max_files) {
+  if (threadIdx.x != 0) return;
+  const uint64_t size = w.vars[V_LISTSZ];
+  const uint64_t nch = (size + kListChunk - 1) / kListChunk;
+  uint32_t run = 0;
+  for (uint64_t ch = 0; ch < nch; ++ch) {
+    const uint32_t v = w.list_chunk[ch];
+    w.list_chunk[ch] = run;
+    run += v;
+  }
+  if (run > max_files) set_err(w, -ENOSPC);
+  w.vars[V_NFILES] = run < max_files ? run : max_files;
+}
+
+// Pass 4: each line start writes its absolute path (relative paths resolve
+// against the list file's directory, R15).
+__global__ void k_grep_list_emit(GrepWork w, const char* dir, uint32_t dir_len, uint32_t max_files) {
+  __shared__ uint32_t warp_tot[32];
+  __shared__ uint32_t base_s;
+  const uint64_t size = w.vars[V_LISTSZ];
+  const uint64_t nch = (size + kListChunk - 1) / kListChunk;
+  const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5, nw = (blockDim.x + 31) / 32;
+  const uint8_t* L = w.list;
+  for (uint64_t ch = blockIdx.x; ch < nch; ch += gridDim.x) {
+    if (tid == 0) base_s = w.list_chunk[ch];
+    __syncthreads();
+    const uint64_t a = ch * kListChunk, b = min(size, a + kListChunk);
+    for (uint64_t t0 = a; t0 < b; t0 += blockDim.x) {
+      const uint64_t i = t0 + tid;
+      const bool start = i < b && line_start(L, i);
+      const uint32_t bal = __ballot_sync(0xFFFFFFFFu, start);
+      if (lane == 0) warp_tot[wid] = __popc(bal);
+      __syncthreads();
+      uint32_t k = base_s;
+      for (int q = 0; q < wid; ++q) k += warp_tot[q];
+      k += __popc(bal & ((1u << lane) - 1));
+      if (start && k < max_files) {
         uint32_t n = 0;
         while (i + n < size && L[i + n] != '\n') ++n;
         char* dst = w.paths + (size_t)k * kMaxPath;
         uint32_t o = 0;
-        if (L[i] != '/') {  // relative to the list file's directory (R15)
+        if (L[i] != '/') {
           for (uint32_t q = 0; q < dir_len && o < kMaxPath - 1; ++q) dst[o++] = dir[q];
           if (o < kMaxPath - 1) dst[o++] = '/';
         }
@@ -208,20 +263,16 @@ __global__ void k_grep_list(const gfs_ctx* c, const char* list_path, const char*
         }
         for (uint32_t q = 0; q < n; ++q) dst[o + q] = (char)L[i + q];
         dst[o + n] = 0;
-        w.path_len[k] = o + n;
-      } else {
-        set_err(w, -ENOSPC);
       }
+      __syncthreads();
+      if (tid == 0) {
+        uint32_t tot = 0;
+        for (int q = 0; q < nw; ++q) tot += warp_tot[q];
+        base_s += tot;
+      }
+      __syncthreads();
     }
-    __syncthreads();
-    if (tid == 0) {
-      uint32_t tot = 0;
-      for (int q = 0; q < (nthr + 31) / 32; ++q) tot += warp_tot[q];
-      base_s += tot;
-    }
-    __syncthreads();
   }
-  if (tid == 0) w.vars[V_NFILES] = base_s < max_files ? base_s : max_files;
 }
 
 // --------------------------------------------------------------- open files
@@ -234,7 +285,8 @@ __global__ void k_grep_open(const gfs_ctx* c, GrepWork w, uint32_t chunk) {
     __syncthreads();
     const uint32_t f = f_s;
     if (f >= nfiles) break;
-    const int fd = gopen(c, w.paths + (size_t)f * kMaxPath, GFS_O_RDONLY);
+    // first gopen of a file goes to the host; page 0 comes back with it
+    const int fd = gopen(c, w.paths + (size_t)f * kMaxPath, GFS_O_RDONLY | GFS_O_PREFETCH);
     const int64_t sz = fd >= 0 ? gfstat_size(c, fd) : fd;
     if (tid == 0) {
       w.fd[f] = fd;
@@ -270,6 +322,10 @@ __global__ void k_grep_plan(GrepWork w) {
       part[q] = run;
       run += v;
     }
+    if (run > w.max_items) {
+      set_err(w, -ENOSPC);
+      run = w.max_items;
+    }
     w.vars[V_NITEMS] = run;
     w.item_base[n] = run;
   }
@@ -279,6 +335,15 @@ __global__ void k_grep_plan(GrepWork w) {
     const uint64_t v = w.item_base[i];
     w.item_base[i] = run;
     run += v;
+  }
+}
+
+// item -> file map (one thread per file)
+__global__ void k_grep_items(GrepWork w) {
+  const uint32_t n = (uint32_t)w.vars[V_NFILES];
+  for (uint32_t f = blockIdx.x * blockDim.x + threadIdx.x; f < n; f += gridDim.x * blockDim.x) {
+    const uint64_t a = w.item_base[f], b = min(w.item_base[f + 1], w.max_items);
+    for (uint64_t i = a; i < b; ++i) w.item_file[i] = f;
   }
 }
 
@@ -297,34 +362,64 @@ __device__ __forceinline__ void pair_add(GrepWork& w, uint32_t f, uint32_t k, ui
   set_err(w, -ENOSPC);
 }
 
+struct ScanAcc {
+  uint64_t dsum, dxor, nh;
+};
+
+// One hit of word k at file position pos: per-item shared count (spilling to
+// the global table when full), digest, optional hit list.
+__device__ __forceinline__ void count_hit(GrepWork& w, uint32_t* ckey, uint32_t* ccnt, uint32_t f, uint32_t k,
+                                          uint64_t pos, uint64_t* hits, uint64_t hit_cap, ScanAcc& acc) {
+  uint32_t cs = (k * 2654435761u) & (kCountSlots - 1);
+  bool done = false;
+  for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & (kCountSlots - 1)) {
+    const uint32_t prev = atomicCAS(&ckey[cs], 0u, k + 1);
+    if (prev == 0 || prev == k + 1) {
+      atomicAdd(&ccnt[cs], 1u);
+      done = true;
+      break;
+    }
+  }
+  if (!done) pair_add(w, f, k, 1);
+  const uint64_t m = hit_mix(f, pos, k);
+  acc.dsum += m;
+  acc.dxor ^= m;
+  ++acc.nh;
+  if (hits) {
+    const unsigned long long idx = atomicAdd(&w.vars[V_NLISTED], 1ull);
+    if (idx < hit_cap) {
+      hits[2 * idx] = ((uint64_t)f << 32) | k;
+      hits[2 * idx + 1] = pos;
+    }
+  }
+}
+
 __global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w, uint32_t chunk, uint64_t* hits,
                                                    uint64_t hit_cap) {
   extern __shared__ __align__(16) uint8_t sm[];
-  uint8_t* buf = sm;                                               // chunk + kPre + kHalo
-  uint32_t* ckey = (uint32_t*)(sm + ((chunk + kPre + kHalo + 15) & ~15u));  // word + 1
+  uint8_t* buf = sm;                                                          // chunk + kPre + kHalo
+  uint32_t* ckey = (uint32_t*)(sm + ((chunk + kPre + kHalo + 15) & ~15u));    // word + 1
   uint32_t* ccnt = ckey + kCountSlots;
+  uint16_t* starts = (uint16_t*)(ccnt + kCountSlots);                         // chunk / 2 token starts
   __shared__ uint64_t item_s;
-  const int tid = threadIdx.x, nthr = blockDim.x;
+  __shared__ uint32_t ntok_s;
+  const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31;
   const uint64_t nitems = w.vars[V_NITEMS];
-  const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
-  uint64_t dsum = 0, dxor = 0, nh = 0;
+  ScanAcc acc{0, 0, 0};
   for (uint32_t i = tid; i < kCountSlots; i += nthr) {  // dynamic smem is not cleared between launches
     ckey[i] = 0;
     ccnt[i] = 0;
   }
   for (;;) {
     __syncthreads();
-    if (tid == 0) item_s = atomicAdd(&w.vars[V_NEXT], 1ull);
+    if (tid == 0) {
+      item_s = atomicAdd(&w.vars[V_NEXT], 1ull);
+      ntok_s = 0;
+    }
     __syncthreads();
     const uint64_t item = item_s;
     if (item >= nitems) break;
-    // file of this item: last f with item_base[f] <= item
-    uint32_t lo = 0, hi = nfiles;
-    while (hi - lo > 1) {
-      const uint32_t mid = (lo + hi) >> 1;
-      if (w.item_base[mid] <= item) lo = mid; else hi = mid;
-    }
-    const uint32_t f = lo;
+    const uint32_t f = w.item_file[item];
     const int fd = w.fd[f];
     const uint64_t size = w.size[f];
     const uint64_t s = (item - w.item_base[f]) * chunk;
@@ -336,63 +431,48 @@ __global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w,
       if (tid == 0) set_err(w, r < 0 ? r : -EIO);
       continue;
     }
-    // positions [s, e) in file coordinates map to buf[pos - ws]
+    // pass 1: compact token starts in [s, e) (file coordinates; buf[pos - ws])
     const uint32_t n_here = (uint32_t)(e - s);
-    for (uint32_t q = tid; q < n_here; q += nthr) {
+    const uint32_t off0 = (uint32_t)(s - ws);
+    for (uint32_t q0 = 0; q0 < n_here; q0 += nthr) {
+      const uint32_t q = q0 + tid;
+      bool st = false;
+      if (q < n_here) {
+        const uint32_t bi = off0 + q;
+        st = is_word(buf[bi]) && (s + q == 0 || !is_word(buf[bi - 1]));
+      }
+      const uint32_t bal = __ballot_sync(0xFFFFFFFFu, st);
+      uint32_t base = 0;
+      if (lane == 0 && bal) base = atomicAdd(&ntok_s, __popc(bal));
+      base = __shfl_sync(0xFFFFFFFFu, base, 0);
+      if (st) starts[base + __popc(bal & ((1u << lane) - 1))] = (uint16_t)q;
+    }
+    __syncthreads();
+    const uint32_t ntok = ntok_s;
+    // pass 2: whole tokens per thread
+    for (uint32_t t = tid; t < ntok; t += nthr) {
+      const uint32_t q = starts[t];
       const uint64_t pos = s + q;
-      const uint32_t bi = (uint32_t)(pos - ws);
-      const uint32_t ch = buf[bi];
-      if (!is_word(ch)) continue;
-      if (pos > 0 && is_word(buf[bi - 1])) continue;
+      const uint32_t bi = off0 + q;
       uint32_t L = 1;
       while (L <= 32 && pos + L < size && is_word(buf[bi + L])) ++L;
       if (L > 32) continue;  // tokens longer than any dictionary word never match
       const uint64_t h = tok_hash(buf + bi, L);
+      const uint64_t want = entry_key(h, L) >> 26;
       uint32_t slot = (uint32_t)h & w.table_mask;
-      const uint64_t want = ((h >> 32) << 32) | ((uint64_t)L << 26);
       for (;;) {
         const uint64_t ent = __ldg((const unsigned long long*)&w.table[slot]);
         if (ent == 0) break;
-        if ((ent >> 26) == (want >> 26)) {
+        if (key_bits(ent) == want) {
           const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
-          const uint8_t* t = w.dict + (size_t)kp * 32;
+          const uint8_t* tw = w.dict + (size_t)kp * 32;
           bool same = true;
-          for (uint32_t i = 0; i < L; ++i) same &= t[i] == buf[bi + i];
+          for (uint32_t i = 0; i < L; ++i) same &= __ldg(tw + i) == buf[bi + i];
           if (same) {
-            uint32_t k = kp;
-            for (;;) {  // the word and its duplicates (each index counts, R14)
-              // per-item count in shared memory; spill to the global table if full
-              uint32_t cs = (k * 2654435761u) & (kCountSlots - 1);
-              bool done = false;
-              for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & (kCountSlots - 1)) {
-                const uint32_t prev = atomicCAS(&ckey[cs], 0u, k + 1);
-                if (prev == 0 || prev == k + 1) {
-                  atomicAdd(&ccnt[cs], 1u);
-                  done = true;
-                  break;
-                }
-              }
-              if (!done) pair_add(w, f, k, 1);
-              const uint64_t m = hit_mix(f, pos, k);
-              dsum += m;
-              dxor ^= m;
-              ++nh;
-              if (hits) {
-                const unsigned long long idx = atomicAdd(&w.vars[V_NLISTED], 1ull);
-                if (idx < hit_cap) {
-                  hits[2 * idx] = ((uint64_t)f << 32) | k;
-                  hits[2 * idx + 1] = pos;
-                }
-              }
-              const uint32_t nx = w.dup_head[k] ? w.dup_head[k] : 0;
-              if (k == kp) {
-                if (!nx) break;
-                k = nx - 1;
-              } else {
-                const uint32_t nn = w.dup_next[k];
-                if (!nn) break;
-                k = nn - 1;
-              }
+            count_hit(w, ckey, ccnt, f, kp, pos, hits, hit_cap, acc);
+            if (ent & kDupBit) {  // the word's duplicates each count (R14)
+              for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
+                count_hit(w, ckey, ccnt, f, d - 1, pos, hits, hit_cap, acc);
             }
             break;
           }
@@ -401,12 +481,11 @@ __global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w,
       }
     }
     __syncthreads();
-    // flush this item's counts: (file, word) table and word totals
+    // flush this item's counts into the (file, word) table
     for (uint32_t i = tid; i < kCountSlots; i += nthr) {
       const uint32_t kk = ckey[i];
       if (kk) {
-        const uint32_t cnt = ccnt[i];
-        pair_add(w, f, kk - 1, cnt);
+        pair_add(w, f, kk - 1, ccnt[i]);
         ckey[i] = 0;
         ccnt[i] = 0;
       }
@@ -414,14 +493,14 @@ __global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w,
   }
   // block-level digest reduction
   for (int o = 16; o; o >>= 1) {
-    dsum += __shfl_xor_sync(0xFFFFFFFFu, dsum, o);
-    dxor ^= __shfl_xor_sync(0xFFFFFFFFu, dxor, o);
-    nh += __shfl_xor_sync(0xFFFFFFFFu, nh, o);
+    acc.dsum += __shfl_xor_sync(0xFFFFFFFFu, acc.dsum, o);
+    acc.dxor ^= __shfl_xor_sync(0xFFFFFFFFu, acc.dxor, o);
+    acc.nh += __shfl_xor_sync(0xFFFFFFFFu, acc.nh, o);
   }
-  if ((tid & 31) == 0) {
-    atomicAdd(&w.vars[V_DSUM], (unsigned long long)dsum);
-    atomicXor(&w.vars[V_DXOR], (unsigned long long)dxor);
-    atomicAdd(&w.vars[V_NHITS], (unsigned long long)nh);
+  if (lane == 0) {
+    atomicAdd(&w.vars[V_DSUM], (unsigned long long)acc.dsum);
+    atomicXor(&w.vars[V_DXOR], (unsigned long long)acc.dxor);
+    atomicAdd(&w.vars[V_NHITS], (unsigned long long)acc.nh);
   }
 }
 
@@ -433,20 +512,29 @@ __global__ void k_grep_close(const gfs_ctx* c, GrepWork w) {
   }
 }
 
-// unique records from the (file, word) table + word totals
+// unique records from the (file, word) table + word totals (warp-aggregated output index)
 __global__ void k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap, uint64_t* totals) {
   const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i <= w.pair_mask; i += stride) {
-    const uint64_t key = w.pair_key[i];
-    if (key == kPairEmpty) continue;
-    const uint64_t cnt = w.pair_cnt[i];
-    const uint32_t k = (uint32_t)key;
-    atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
-    const unsigned long long idx = atomicAdd(&w.vars[V_NREC], 1ull);
-    if (idx < rec_cap) {
-      rec[3 * idx] = (uint32_t)(key >> 32);
-      rec[3 * idx + 1] = k;
-      rec[3 * idx + 2] = (uint32_t)cnt;
+  const int lane = threadIdx.x & 31;
+  const uint64_t n = w.pair_mask + 1;
+  for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x; i0 < n; i0 += stride) {
+    const uint64_t i = i0 + threadIdx.x;
+    const uint64_t key = i < n ? w.pair_key[i] : kPairEmpty;
+    const bool v = key != kPairEmpty;
+    const uint32_t bal = __ballot_sync(0xFFFFFFFFu, v);
+    unsigned long long base = 0;
+    if (lane == 0 && bal) base = atomicAdd(&w.vars[V_NREC], (unsigned long long)__popc(bal));
+    base = __shfl_sync(0xFFFFFFFFu, base, 0);
+    if (v) {
+      const uint64_t cnt = w.pair_cnt[i];
+      const uint32_t k = (uint32_t)key;
+      atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
+      const uint64_t idx = base + __popc(bal & ((1u << lane) - 1));
+      if (idx < rec_cap) {
+        rec[3 * idx] = (uint32_t)(key >> 32);
+        rec[3 * idx + 1] = k;
+        rec[3 * idx + 2] = (uint32_t)cnt;
+      }
     }
   }
 }
@@ -490,34 +578,42 @@ uint64_t pow2_at_least(uint64_t x) {
 struct Layout {
   uint64_t off[16];
   uint64_t total;
+  uint64_t max_items;
 };
 
 Layout layout(const gfs_grep_params* p) {
   Layout L{};
   const uint64_t tcap = pow2_at_least(p->max_words * 2ull < 1024 ? 1024 : p->max_words * 2ull);
   const uint64_t pcap = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap);
+  // items: one per chunk of corpus plus one partial chunk per file
+  L.max_items = p->corpus_cap / (p->chunk ? p->chunk : 1) + p->max_files + 1;
   const uint64_t sizes[] = {
-      (uint64_t)p->max_words * 32,         // dict
-      tcap * 8,                            // table
-      (uint64_t)p->max_words * 4,          // dup_head
-      (uint64_t)p->max_words * 4,          // dup_next
-      p->list_cap + 64,                    // list
-      (uint64_t)p->max_files * kMaxPath,   // paths
-      (uint64_t)p->max_files * 4,          // path_len
-      (uint64_t)p->max_files * 4,          // fd
-      (uint64_t)p->max_files * 8,          // size
-      ((uint64_t)p->max_files + 1) * 8,    // item_base
-      pcap * 8,                            // pair_key
-      pcap * 8,                            // pair_cnt
-      V_NVARS * 8,                         // vars
+      (uint64_t)p->max_words * 32,                         // dict
+      tcap * 8,                                            // table
+      (uint64_t)p->max_words * 4,                          // dup_head
+      (uint64_t)p->max_words * 4,                          // dup_next
+      p->list_cap + 64,                                    // list
+      (p->list_cap / kListChunk + 2) * 4,                  // list_chunk
+      (uint64_t)p->max_files * kMaxPath,                   // paths
+      (uint64_t)p->max_files * 4,                          // fd
+      (uint64_t)p->max_files * 8,                          // size
+      ((uint64_t)p->max_files + 1) * 8,                    // item_base
+      L.max_items * 4,                                     // item_file
+      pcap * 8,                                            // pair_key
+      pcap * 8,                                            // pair_cnt
+      V_NVARS * 8,                                         // vars
   };
   uint64_t o = 0;
-  for (int i = 0; i < 13; ++i) {
+  for (int i = 0; i < 14; ++i) {
     L.off[i] = o;
     o += (sizes[i] + 255) & ~255ull;
   }
   L.total = o;
   return L;
+}
+
+uint32_t scan_smem(uint32_t chunk) {
+  return ((chunk + kPre + kHalo + 15) & ~15u) + 2 * kCountSlots * 4 + (chunk / 2 + 16) * 2;
 }
 
 }  // namespace
@@ -528,8 +624,8 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
                      const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
                      uint64_t* d_hits, uint64_t* d_summary) {
   if (!h || !dict_path || !list_path || !p || !d_work || !d_totals || !d_summary || p->max_files == 0 ||
-      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) || p->grid == 0 ||
-      p->block == 0 || p->block > 256 || (p->block & 31))
+      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) || p->chunk > 65536 ||
+      p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31))
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
   const Layout L = layout(p);
@@ -541,15 +637,17 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   w.dup_head = (uint32_t*)(base + L.off[2]);
   w.dup_next = (uint32_t*)(base + L.off[3]);
   w.list = base + L.off[4];
-  w.paths = (char*)(base + L.off[5]);
-  w.path_len = (uint32_t*)(base + L.off[6]);
+  w.list_chunk = (uint32_t*)(base + L.off[5]);
+  w.paths = (char*)(base + L.off[6]);
   w.fd = (int32_t*)(base + L.off[7]);
   w.size = (uint64_t*)(base + L.off[8]);
   w.item_base = (uint64_t*)(base + L.off[9]);
-  w.pair_key = (uint64_t*)(base + L.off[10]);
-  w.pair_cnt = (uint64_t*)(base + L.off[11]);
+  w.item_file = (uint32_t*)(base + L.off[10]);
+  w.max_items = L.max_items;
+  w.pair_key = (uint64_t*)(base + L.off[11]);
+  w.pair_cnt = (uint64_t*)(base + L.off[12]);
   w.pair_mask = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap) - 1;
-  w.vars = (unsigned long long*)(base + L.off[12]);
+  w.vars = (unsigned long long*)(base + L.off[13]);
 
   // staged strings: dict path, list path, list directory
   static char* d_str = nullptr;
@@ -580,31 +678,39 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   cudaEventRecord(ev, s);
 
   const gfs_ctx* c = gfs_device_ctx(h);
-  const uint32_t smem = ((p->chunk + kPre + kHalo + 15) & ~15u) + 2 * kCountSlots * 4;
+  const uint32_t smem = scan_smem(p->chunk);
   if (smem > 227 * 1024) return -EINVAL;
   cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-  // GFS_GREP_DEBUG=1: synchronise after each stage and report the first failing one
+  // GFS_GREP_DEBUG=1: synchronise after each stage, print its time and the first error
   const bool dbg = getenv("GFS_GREP_DEBUG") && *getenv("GFS_GREP_DEBUG") == '1';
+  struct timespec ts_prev;
+  clock_gettime(CLOCK_MONOTONIC, &ts_prev);
   auto stage = [&](const char* name) {
     if (!dbg) return;
     cudaError_t e = cudaStreamSynchronize(s);
-    long long err = 0;
-    cudaMemcpy(&err, &w.vars[V_ERR], 8, cudaMemcpyDeviceToHost);
+    struct timespec ts;
+    clock_gettime(CLOCK_MONOTONIC, &ts);
     unsigned long long v[V_NVARS];
     cudaMemcpy(v, w.vars, sizeof(v), cudaMemcpyDeviceToHost);
-    fprintf(stderr, "gfs_grep[%s]: cuda=%s err=%lld nfiles=%llu nwords=%llu nitems=%llu bytes=%llu\n", name,
-            cudaGetErrorString(e), err, v[V_NFILES], v[V_NWORDS], v[V_NITEMS], v[V_BYTES]);
+    fprintf(stderr, "gfs_grep[%s]: %.3f ms cuda=%s err=%lld nfiles=%llu nwords=%llu nitems=%llu bytes=%llu\n", name,
+            (ts.tv_sec - ts_prev.tv_sec) * 1e3 + (ts.tv_nsec - ts_prev.tv_nsec) * 1e-6, cudaGetErrorString(e),
+            (long long)v[V_ERR], v[V_NFILES], v[V_NWORDS], v[V_NITEMS], v[V_BYTES]);
+    ts_prev = ts;
   };
+  const uint64_t lb = p->list_cap / kListChunk + 1;
+  const uint32_t list_blocks = (uint32_t)(lb < 1024 ? lb : 1024);
   k_grep_init<<<1024, 256, 0, s>>>(w, p->max_words);
-  const uint32_t dict_blocks = 64;
-  k_grep_dict<<<dict_blocks, 256, 0, s>>>(c, d_str, w, p->max_words);
+  k_grep_dict<<<64, 256, 0, s>>>(c, d_str, w, p->max_words);
   stage("dict");
-  k_grep_list<<<1, 256, 0, s>>>(c, d_str + kMaxPath, d_str + 2 * kMaxPath, (uint32_t)dl, w, p->list_cap,
-                                 p->max_files);
+  k_grep_list_read<<<list_blocks, 256, 0, s>>>(c, d_str + kMaxPath, w, p->list_cap);
+  k_grep_list_count<<<list_blocks, 256, 0, s>>>(w);
+  k_grep_list_scan<<<1, 32, 0, s>>>(w, p->max_files);
+  k_grep_list_emit<<<list_blocks, 256, 0, s>>>(w, d_str + 2 * kMaxPath, (uint32_t)dl, p->max_files);
   stage("list");
   k_grep_open<<<p->grid, 128, 0, s>>>(c, w, p->chunk);
   stage("open");
   k_grep_plan<<<1, 1024, 0, s>>>(w);
+  k_grep_items<<<256, 256, 0, s>>>(w);
   k_grep_scan<<<p->grid, p->block, smem, s>>>(c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0);
   stage("scan");
   if (!p->keep_open) k_grep_close<<<p->grid, 32, 0, s>>>(c, w);

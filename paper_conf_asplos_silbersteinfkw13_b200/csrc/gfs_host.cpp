@@ -28,14 +28,17 @@
 #include <cstdio>
 #include <cstdlib>
 #include <cstring>
+#include <deque>
 #include <fcntl.h>
 #include <mutex>
 #include <sched.h>
 #include <string>
 #include <sys/mman.h>
+#include <sys/resource.h>
 #include <sys/stat.h>
 #include <thread>
 #include <unistd.h>
+#include <unordered_map>
 #include <vector>
 
 #include <cuda_runtime.h>
@@ -146,20 +149,37 @@ struct VersionTable {
 
 enum {
   HS_RPC = 0, HS_READ, HS_WRITE, HS_OPEN, HS_CLOSE, HS_TRUNC, HS_BYTES_H2D, HS_BYTES_D2H, HS_PREAD_NS,
-  HS_ERRORS, HS_MERGES, HS_N
+  HS_ERRORS, HS_MERGES, HS_BUSY_NS, HS_OPEN_NS, HS_OPEN_SYS_NS, HS_OPEN_PF_NS, HS_OPEN_TAB_NS, HS_N
 };
 
 }  // namespace
 
+// One host file the GPU knows by its hfid (metadata only). Each daemon worker
+// has a PRIVATE fd table (unshare(CLONE_FILES)): open()/close() in one
+// process serialise on its fd-table lock, so workers sharing a table open
+// files slower than one thread does. A worker re-opens a file by path the
+// first time it serves it (the (dev, ino) check turns a replaced file into
+// -ESTALE); `gen` invalidates cached fds when an hfid is recycled.
 struct HostFile {
-  int fd = -1;
+  bool live = false;
+  uint32_t gen = 0;
   uint32_t mode = 0;
   uint64_t dev = 0, ino = 0;
+  std::string path;
+};
+
+struct WorkerFd {
+  int fd;
+  uint32_t gen;
 };
 
 struct Worker {
   std::thread th;
   std::vector<uint8_t> merge;
+  std::unordered_map<uint32_t, WorkerFd> fds;        // hfid -> fd in this worker's table
+  std::deque<uint32_t> fifo;                          // eviction order of fds
+  std::unordered_map<std::string, int> dirfds;       // directory fds for openat()
+  size_t cap = 1024;
 };
 
 struct gfs_handle {
@@ -176,9 +196,10 @@ struct gfs_handle {
   std::vector<Worker> workers;
   std::atomic<uint64_t> next_ticket{0};
   std::atomic<bool> running{false};
-  std::mutex fd_mu;
+  std::mutex fd_mu;  // protects files / free_hfids
   std::vector<HostFile> files;
   std::vector<uint32_t> free_hfids;
+  size_t fd_cap = 1024;  // per worker
   VersionTable vt;
   std::atomic<uint64_t> hs[HS_N];
 };
@@ -201,30 +222,104 @@ int cuda_err(cudaError_t e) {
     }                                 \
   } while (0)
 
-uint32_t alloc_hfid(gfs_handle* h, const HostFile& f) {
+uint32_t alloc_hfid(gfs_handle* h, HostFile f) {
   std::lock_guard<std::mutex> g(h->fd_mu);
+  f.live = true;
+  uint32_t id;
   if (!h->free_hfids.empty()) {
-    uint32_t id = h->free_hfids.back();
+    id = h->free_hfids.back();
     h->free_hfids.pop_back();
+    f.gen = h->files[id].gen;
     h->files[id] = f;
-    return id;
+  } else {
+    f.gen = 0;
+    h->files.push_back(f);
+    id = (uint32_t)(h->files.size() - 1);
   }
-  h->files.push_back(f);
-  return (uint32_t)(h->files.size() - 1);
+  return id;
 }
 
-HostFile get_hfid(gfs_handle* h, uint32_t id) {
+// Metadata of a live hfid.
+bool hfid_meta(gfs_handle* h, uint32_t id, HostFile* out) {
   std::lock_guard<std::mutex> g(h->fd_mu);
-  if (id >= h->files.size()) return HostFile();
-  return h->files[id];
+  if (id >= h->files.size() || !h->files[id].live) return false;
+  *out = h->files[id];
+  return true;
 }
 
 void free_hfid(gfs_handle* h, uint32_t id) {
   std::lock_guard<std::mutex> g(h->fd_mu);
-  if (id >= h->files.size() || h->files[id].fd < 0) return;
-  ::close(h->files[id].fd);
+  if (id >= h->files.size() || !h->files[id].live) return;
+  const uint32_t gen = h->files[id].gen + 1;
   h->files[id] = HostFile();
+  h->files[id].gen = gen;  // cached fds of the old file are now stale
   h->free_hfids.push_back(id);
+}
+
+// open(path) as openat(this worker's cached fd of dirname(path), basename).
+int w_open_path(Worker& w, const std::string& path, int flags) {
+  const size_t slash = path.rfind('/');
+  if (slash == std::string::npos || slash == 0) return ::open(path.c_str(), flags, 0644);
+  const std::string dir = path.substr(0, slash);
+  auto it = w.dirfds.find(dir);
+  int dfd;
+  if (it != w.dirfds.end()) {
+    dfd = it->second;
+  } else {
+    dfd = ::open(dir.c_str(), O_RDONLY | O_DIRECTORY | O_PATH);
+    if (dfd < 0) return ::open(path.c_str(), flags, 0644);
+    if (w.dirfds.size() > 4096) {  // bound the directory cache
+      for (auto& kv : w.dirfds) ::close(kv.second);
+      w.dirfds.clear();
+    }
+    w.dirfds.emplace(dir, dfd);
+  }
+  return ::openat(dfd, path.c_str() + slash + 1, flags, 0644);
+}
+
+void w_make_room(Worker& w) {
+  while (w.fds.size() >= w.cap && !w.fifo.empty()) {
+    const uint32_t id = w.fifo.front();
+    w.fifo.pop_front();
+    auto it = w.fds.find(id);
+    if (it != w.fds.end()) {
+      ::close(it->second.fd);
+      w.fds.erase(it);
+    }
+  }
+}
+
+void w_cache(Worker& w, uint32_t id, int fd, uint32_t gen) {
+  auto it = w.fds.find(id);
+  if (it != w.fds.end()) {
+    ::close(it->second.fd);
+    it->second = WorkerFd{fd, gen};
+    return;
+  }
+  w_make_room(w);
+  w.fds.emplace(id, WorkerFd{fd, gen});
+  w.fifo.push_back(id);
+}
+
+// This worker's fd for hfid (opened by path on first use). -errno on failure.
+int w_fd(gfs_handle* h, Worker& w, uint32_t id) {
+  HostFile m;
+  if (!hfid_meta(h, id, &m)) return -EBADF;
+  auto it = w.fds.find(id);
+  if (it != w.fds.end()) {
+    if (it->second.gen == m.gen) return it->second.fd;
+    ::close(it->second.fd);  // the hfid was recycled for another file
+    w.fds.erase(it);
+  }
+  const int fd = w_open_path(w, m.path, (m.mode & GFS_O_GWRONCE) ? O_RDWR : O_RDONLY);
+  if (fd < 0) return -errno;
+  struct stat st;
+  if (fstat(fd, &st) != 0 || (uint64_t)st.st_dev != m.dev || (uint64_t)st.st_ino != m.ino) {
+    ::close(fd);
+    return -ESTALE;
+  }
+  w_cache(w, id, fd, m.gen);
+  return fd;
 }
 
 inline void complete(gfs_handle* h, uint32_t slot, uint64_t ticket, int32_t result) {
@@ -235,11 +330,17 @@ inline uint8_t* staging_slot(gfs_handle* h, uint32_t stage) {
   return h->staging_h + ((size_t)stage << h->h.page_shift);
 }
 
-int32_t do_open(gfs_handle* h, uint32_t slot, const gfs_rpc_req& q) {
+int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
+  auto tk0 = std::chrono::steady_clock::now();
+  auto lap = [&](int k) {
+    const auto t = std::chrono::steady_clock::now();
+    h->hs[k] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(t - tk0).count();
+    tk0 = t;
+  };
   gfs_rpc_resp* rs = h->resp_h + slot;
   std::string path(h->paths_h + (size_t)slot * GFS_MAX_PATH, q.path_len < GFS_MAX_PATH ? q.path_len : 0);
   const bool gw = (q.flags & GFS_O_GWRONCE) != 0;
-  int fd = ::open(path.c_str(), gw ? (O_RDWR | O_CREAT) : O_RDONLY, 0644);
+  int fd = w_open_path(w, path, gw ? (O_RDWR | O_CREAT) : O_RDONLY);
   if (fd < 0) {
     rs->status = -errno;
     return rs->status;
@@ -250,27 +351,45 @@ int32_t do_open(gfs_handle* h, uint32_t slot, const gfs_rpc_req& q) {
     ::close(fd);
     return rs->status;
   }
+  lap(HS_OPEN_SYS_NS);
+  // OPEN with prefetch: page 0 comes back with the reply (one RPC per small file)
+  rs->pad[0] = 0;
+  if (q.stage != 0xFFFFFFFFu && !gw && q.stage < h->h.staging_slots && st.st_size > 0) {
+    const uint64_t n = (uint64_t)st.st_size < h->h.page_size ? (uint64_t)st.st_size : h->h.page_size;
+    uint8_t* buf = staging_slot(h, q.stage);
+    const int64_t r = pread_full(fd, buf, n, 0);
+    if (r >= 0) {
+      if ((uint64_t)r < n) memset(buf + r, 0, n - (size_t)r);
+      rs->pad[0] = n;
+      h->hs[HS_READ]++;
+      h->hs[HS_BYTES_H2D] += n;
+    }
+  }
+  lap(HS_OPEN_PF_NS);
   uint32_t hfid;
   bool reused = false;
-  if (q.arg) {  // re-open of a cached file: keep its host fd if it is the same file
+  if (q.arg) {  // re-open of a cached file: keep its hfid if it is the same file
     const uint32_t old = (uint32_t)(q.arg - 1);
-    HostFile of = get_hfid(h, old);
-    if (of.fd >= 0 && of.dev == (uint64_t)st.st_dev && of.ino == (uint64_t)st.st_ino &&
+    HostFile of;
+    if (hfid_meta(h, old, &of) && of.dev == (uint64_t)st.st_dev && of.ino == (uint64_t)st.st_ino &&
         (of.mode & GFS_O_GWRONCE) >= (q.flags & GFS_O_GWRONCE)) {
-      ::close(fd);
       hfid = old;
       reused = true;
+      w_cache(w, hfid, fd, of.gen);
     } else {
       free_hfid(h, old);
     }
   }
   if (!reused) {
     HostFile f;
-    f.fd = fd;
     f.mode = q.flags;
     f.dev = st.st_dev;
     f.ino = st.st_ino;
+    f.path = path;
     hfid = alloc_hfid(h, f);
+    HostFile m;
+    if (hfid_meta(h, hfid, &m)) w_cache(w, hfid, fd, m.gen);
+    else ::close(fd);
   }
   rs->size = (int64_t)st.st_size;
   rs->version = h->vt.get(st.st_dev, st.st_ino);
@@ -280,16 +399,17 @@ int32_t do_open(gfs_handle* h, uint32_t slot, const gfs_rpc_req& q) {
   rs->hfid = hfid;
   rs->status = 0;
   h->hs[HS_OPEN]++;
+  lap(HS_OPEN_TAB_NS);
   return 0;
 }
 
-int32_t do_read(gfs_handle* h, const gfs_rpc_req& q) {
-  HostFile f = get_hfid(h, q.hfid);
-  if (f.fd < 0) return -EBADF;
+int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   if (q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
+  const int fd = w_fd(h, w, q.hfid);
+  if (fd < 0) return fd;
   uint8_t* buf = staging_slot(h, q.stage);
   auto t0 = std::chrono::steady_clock::now();
-  int64_t n = pread_full(f.fd, buf, q.len, q.file_off);
+  int64_t n = pread_full(fd, buf, q.len, q.file_off);
   h->hs[HS_PREAD_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
                             std::chrono::steady_clock::now() - t0).count();
   if (n < 0) return (int32_t)n;
@@ -300,22 +420,24 @@ int32_t do_read(gfs_handle* h, const gfs_rpc_req& q) {
 }
 
 int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
-  HostFile f = get_hfid(h, q.hfid);
-  if (f.fd < 0) return -EBADF;
+  HostFile f;
+  if (!hfid_meta(h, q.hfid, &f)) return -EBADF;
   if (!(f.mode & GFS_O_GWRONCE)) return -EBADF;  // read-only files are never written back
   const uint64_t in_page = q.file_off & (h->h.page_size - 1);
   if (in_page + q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
+  const int fd = w_fd(h, w, q.hfid);
+  if (fd < 0) return fd;
   uint8_t* buf = staging_slot(h, q.stage) + in_page;
   if (!(q.flags & GFS_WF_FULL)) {
     // Not every byte of the range was written: diff against zeros.
     w.merge.assign(q.len, 0);
-    int64_t r = pread_full(f.fd, w.merge.data(), q.len, q.file_off);
+    int64_t r = pread_full(fd, w.merge.data(), q.len, q.file_off);
     if (r < 0) return (int32_t)r;
     for (uint32_t i = 0; i < q.len; ++i)
       if (buf[i] == 0) buf[i] = w.merge[i];
     h->hs[HS_MERGES]++;
   }
-  int64_t r = pwrite_full(f.fd, buf, q.len, q.file_off);
+  int64_t r = pwrite_full(fd, buf, q.len, q.file_off);
   if (r < 0) return (int32_t)r;
   h->vt.bump(f.dev, f.ino);
   h->hs[HS_WRITE]++;
@@ -325,6 +447,10 @@ int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
 
 void worker_loop(gfs_handle* h, int wi) {
   Worker& w = h->workers[wi];
+  w.cap = h->fd_cap;
+  // A private fd table for this worker (see HostFile): its open()/close()
+  // no longer contend with the other workers' on one table lock.
+  unshare(CLONE_FILES);
   const uint32_t R = h->h.ring_slots;
   while (h->running.load(std::memory_order_acquire)) {
     const uint64_t t = h->next_ticket.fetch_add(1);
@@ -358,18 +484,24 @@ void worker_loop(gfs_handle* h, int wi) {
     q.path_len = vq->path_len;
     q.stage = vq->stage;
     int32_t res;
+    const auto tb = std::chrono::steady_clock::now();
     switch (q.op) {
-      case GFS_OP_READ: res = do_read(h, q); break;
+      case GFS_OP_READ: res = do_read(h, w, q); break;
       case GFS_OP_WRITE: res = do_write(h, w, q); break;
-      case GFS_OP_OPEN: res = do_open(h, slot, q); break;
+      case GFS_OP_OPEN:
+        res = do_open(h, w, slot, q);
+        h->hs[HS_OPEN_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
+                                 std::chrono::steady_clock::now() - tb).count();
+        break;
       case GFS_OP_CLOSE:
         free_hfid(h, q.hfid);
         h->hs[HS_CLOSE]++;
         res = 0;
         break;
       case GFS_OP_TRUNC: {
-        HostFile f = get_hfid(h, q.hfid);
-        res = f.fd < 0 ? -EBADF : (ftruncate(f.fd, (off_t)q.arg) == 0 ? 0 : -errno);
+        HostFile f;
+        const int fd = hfid_meta(h, q.hfid, &f) ? w_fd(h, w, q.hfid) : -EBADF;
+        res = fd < 0 ? fd : (ftruncate(fd, (off_t)q.arg) == 0 ? 0 : -errno);
         if (res == 0) h->vt.bump(f.dev, f.ino);
         h->hs[HS_TRUNC]++;
         break;
@@ -380,7 +512,14 @@ void worker_loop(gfs_handle* h, int wi) {
     if (res < 0) h->hs[HS_ERRORS]++;
     h->hs[HS_RPC]++;
     complete(h, slot, t, res);
+    h->hs[HS_BUSY_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
+                             std::chrono::steady_clock::now() - tb).count();
   }
+  for (auto& kv : w.fds) ::close(kv.second.fd);  // this worker's private table
+  for (auto& kv : w.dirfds) ::close(kv.second);
+  w.fds.clear();
+  w.fifo.clear();
+  w.dirfds.clear();
 }
 
 void free_all(gfs_handle* h) {
@@ -398,8 +537,6 @@ void free_all(gfs_handle* h) {
   if (h->cpl_h) cudaFreeHost(h->cpl_h);
   if (h->staging_h) cudaFreeHost(h->staging_h);
   if (h->priv) cudaStreamDestroy(h->priv);
-  for (auto& f : h->files)
-    if (f.fd >= 0) ::close(f.fd);
   h->vt.close();
 }
 
@@ -435,8 +572,24 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev == 0) return -ENODEV;
   if (cfg->device < 0 || cfg->device >= ndev) return -ENODEV;
 
+  {  // the daemon keeps one host fd per cached file (a source tree is ~30k files)
+    struct rlimit rl;
+    if (getrlimit(RLIMIT_NOFILE, &rl) == 0 && rl.rlim_cur < rl.rlim_max) {
+      rl.rlim_cur = rl.rlim_max;
+      setrlimit(RLIMIT_NOFILE, &rl);
+    }
+  }
   gfs_handle* h = new gfs_handle();
   for (auto& x : h->hs) x = 0;
+  {
+    struct rlimit rl;
+    const uint64_t lim = getrlimit(RLIMIT_NOFILE, &rl) == 0 ? (uint64_t)rl.rlim_cur : 1024;
+    const uint64_t want = lim * 3 / 4;  // leave room for the application and other handles
+    const uint64_t cap = want > 65536 ? 65536 : want;
+    h->fd_cap = cap < 64 ? 64 : cap;
+    const char* env = getenv("GFS_FD_CAP");  // tests: force fd-cache eviction
+    if (env && atoi(env) > 0) h->fd_cap = (size_t)atoi(env);
+  }
   h->cfg = *cfg;
   int rc = 0;
   gfs_ctx& c = h->h;

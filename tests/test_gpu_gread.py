@@ -107,7 +107,12 @@ def test_locked_traversal_same_bytes(g, shmdir, locked):
     with _fs(g, cache_bytes=1024 * P, page_size=P, flags=locked) as fs:
         ret, dst, dstoff = fs.gread_calls(path, offs, lens, grid=48)
         st = fs.stats()
-    check_calls(path, size, offs, lens, ret, dst, dstoff)
+        hs = fs.host_stats()
+        info = fs.info()
+    try:
+        check_calls(path, size, offs, lens, ret, dst, dstoff)
+    except AssertionError as e:
+        raise AssertionError(f"{e} | dev {st} | host {hs} | info {info}")
     if locked:
         assert st["locked"] > 0 and st["lockfree"] == 0
     else:

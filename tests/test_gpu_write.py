@@ -131,3 +131,25 @@ def test_gftruncate(g, shmdir):
         fs.gwrite_calls(path, [0], [3], b"abc")
         assert fs.gfsync(path) == 0
     assert host(path) == b"abc"
+
+
+def test_more_files_than_fd_cache(g, shmdir):
+    """The daemon's fd cache closes idle host fds and re-opens them by path."""
+    paths = []
+    for i in range(300):
+        p = os.path.join(shmdir, f"f{i}.bin")
+        open(p, "wb").write(bytes([i % 251 + 1]) * (100 + i))
+        paths.append(p)
+    os.environ["GFS_FD_CAP"] = "64"  # read at gfs_init: at most 64 host fds open
+    try:
+        with g.GpuFS(cache_bytes=64 << 20, page_size=4096, timeout_ms=30000, daemon_threads=2) as fs:
+            for rep in range(2):
+                for i in (0, 150, 299, 7):
+                    pins = [fs.pin(p) for p in paths]  # 300 files open on the GPU at once
+                    assert min(pins) >= 0
+                    ret, d, _ = fs.gread_calls(paths[i], [0], [1000], grid=1)
+                    assert ret[0] == 100 + i and d[:100 + i].tobytes() == bytes([i % 251 + 1]) * (100 + i)
+                    for fd in pins:
+                        assert fs.unpin(fd) == 0
+    finally:
+        del os.environ["GFS_FD_CAP"]
