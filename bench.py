@@ -440,9 +440,9 @@ def main():
     ap.add_argument("--daemon-threads", type=int, default=12)
     ap.add_argument("--hit-file-gib", type=int, default=4)
     ap.add_argument("--hit-page-kib", type=int, default=512)
-    ap.add_argument("--hit-grid", type=int, default=592)
-    ap.add_argument("--hit-block", type=int, default=256)
-    ap.add_argument("--hit-calls", type=int, default=2048)
+    ap.add_argument("--hit-grid", type=int, default=1184)   # 8 blocks/SM: lookups of one block overlap
+    ap.add_argument("--hit-block", type=int, default=128)   # copies of the others (measured best)
+    ap.add_argument("--hit-calls", type=int, default=1024)
     ap.add_argument("--ref-sample-mib", type=int, default=2048)
     ap.add_argument("--timeout-ms", type=int, default=60000)
     ap.add_argument("--no-hit", action="store_true")
