@@ -175,6 +175,20 @@ int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* lis
              const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
              uint64_t* d_hits, uint64_t* d_summary);
 
+/* --------------------------------------------------------------------------
+ * Out-of-core fp32 matrix-vector product (§5.1.4): y = A x with
+ * A a row-major little-endian fp32 file (rows x cols), x a cols-long fp32
+ * file, y written to y_path through gftruncate + gwrite + gfsync (O_GWRONCE).
+ * A is consumed through gmmap page by page; products accumulate in fp64 and
+ * each y_r is rounded to fp32 once. d_x: device scratch of cols floats (x is
+ * gread into it). d_y: optional device copy of y (rows floats). *d_err:
+ * 0 or the most negative error. Needs ceil(rows/grid)*4 <= 160 KiB (y slice
+ * of a block in shared memory).
+ * ------------------------------------------------------------------------ */
+int gfs_matvec(gfs_handle* h, void* stream, const char* a_path, const char* x_path, const char* y_path,
+               uint64_t rows, uint64_t cols, float* d_x, float* d_y, int64_t* d_err, uint32_t grid,
+               uint32_t block);
+
 #ifdef __cplusplus
 }
 #endif

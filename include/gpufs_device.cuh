@@ -542,7 +542,8 @@ __device__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t h
   const uint64_t page = ld_rlx64(&c->f_tag[f]) & 0xFFFFFFFFull;
   const int st = stage_alloc(c);
   if (st < 0) return st;
-  block_copy_plain(stage_ptr(c, st) + lo, frame_ptr(c, f) + lo, hi - lo, 0, 1);
+  // frame bytes via L2 (.cg): this SM's L1 may hold lines of a previous tenant
+  block_copy_from_frame(stage_ptr(c, st) + lo, frame_ptr(c, f) + lo, hi - lo, 0, 1);
   __threadfence_system();
   const int32_t r = rpc_call(c, GFS_OP_WRITE, hfid, (page << c->page_shift) + lo, st, hi - lo,
                              wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, nullptr);
@@ -678,6 +679,22 @@ __device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs,
   }
   red_add_rlx(&c->f_state[f], 0xFFFFFFFFu);
   return -1;
+}
+
+// True if page `page` is installed and currently FILLING or EVICTING (no
+// reference taken, no lock): a waiter can keep waiting without contending.
+__device__ __forceinline__ bool peek_busy(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
+  uint32_t node = fs.root;
+  for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
+    node = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
+    if (!node) return false;
+  }
+  const uint32_t s = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
+  if (!s) return false;
+  const uint32_t f = s - 1;
+  const uint32_t st = ld_rlx(&c->f_state[f]);
+  return (st & (GFS_ST_FILLING | GFS_ST_EVICTING)) &&
+         ld_rlx64(&c->f_tag[f]) == (((uint64_t)fs.uid << 32) | (uint32_t)page);
 }
 
 struct Lk {
@@ -818,8 +835,14 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
   for (int round = 0;; ++round) {
     if (!(first_done && round == 0)) {
       if (tid < (int)cnt && sc.frame[tid] == kBusy) {
-        int f = fast ? lookup_fast(c, fs, pb + tid) : -1;
-        if (f >= 0) {
+        // Retries of busy pages always try the lock-free path first: in the
+        // locked ablation, hundreds of lanes re-taking the file lock while
+        // they wait starve the lanes that still have to install pages.
+        int f = (fast || round > 0) ? lookup_fast(c, fs, pb + tid) : -1;
+        if (f < 0 && round > 0 && peek_busy(c, fs, pb + tid)) {
+          // still being filled/evicted elsewhere: look again later without
+          // taking the lock (lock-taking retries starve the installers)
+        } else if (f >= 0) {
           sc.frame[tid] = f;
           sc.fill[tid] = 0;
           sc.stage[tid] = -1;
@@ -1450,7 +1473,7 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
       __syncthreads();
       for (uint32_t i = 0; i < cnt; ++i)
         if (sc.frame[i] >= 0)
-          block_copy_plain(stage_ptr(c, sc.stage[i]) + sc.lo[i], frame_ptr(c, (uint32_t)sc.frame[i]) + sc.lo[i],
+          block_copy_from_frame(stage_ptr(c, sc.stage[i]) + sc.lo[i], frame_ptr(c, (uint32_t)sc.frame[i]) + sc.lo[i],
                            sc.hi[i] - sc.lo[i], tid, nthr);
       __threadfence_system();
       __syncthreads();

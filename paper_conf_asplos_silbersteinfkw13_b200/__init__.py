@@ -82,6 +82,7 @@ def lib():
             "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
             "gfs_grep_work_bytes": ([ctypes.POINTER(gfs_grep_params)], U64),
             "gfs_grep": ([P, P, CS, CS, ctypes.POINTER(gfs_grep_params), P, P, U64, P, P, P], I),
+            "gfs_matvec": ([P, P, CS, CS, CS, U64, U64, P, P, P, U32, U32], I),
         }
         for name, (args, res) in sig.items():
             fn = getattr(L, name)
@@ -184,6 +185,11 @@ def gfs_grep(h, stream, dict_path, list_path, p: gfs_grep_params, d_work, d_rec,
              d_summary):
     return _ck(lib().gfs_grep(h, stream, _b(dict_path), _b(list_path), ctypes.byref(p), d_work, d_rec, rec_cap,
                               d_totals, d_hits, d_summary), "gfs_grep")
+
+
+def gfs_matvec(h, stream, a_path, x_path, y_path, rows, cols, d_x, d_y, d_err, grid, block):
+    return _ck(lib().gfs_matvec(h, stream, _b(a_path), _b(x_path), _b(y_path), rows, cols, d_x, d_y, d_err, grid,
+                                block), "gfs_matvec")
 
 
 from . import build  # noqa: E402,F401

@@ -227,6 +227,28 @@ class GpuFS:
         out["state"] = state
         return out
 
+    # mat-vec -------------------------------------------------------------------
+    def matvec(self, a_path, x_path, y_path, rows, cols, grid=None, block=256, stream=None, sync=True, state=None):
+        """y = A x through gmmap/gwrite/gfsync. Returns (y device tensor, err)."""
+        torch = _torch()
+        from . import gfs_matvec
+        dev = f"cuda:{self.device}"
+        if grid is None:
+            grid = max(1, min(rows, 4 * 148))
+            while (rows + grid - 1) // grid * 4 > 160 * 1024:
+                grid *= 2
+        if state is None:
+            state = dict(x=torch.empty(cols, dtype=torch.float32, device=dev),
+                         y=torch.empty(rows, dtype=torch.float32, device=dev),
+                         err=torch.zeros(2, dtype=torch.int64, device=dev))
+        s, sp = self._stream(stream)
+        gfs_matvec(self.h, sp, a_path, x_path, y_path, rows, cols, state["x"].data_ptr(), state["y"].data_ptr(),
+                   state["err"].data_ptr(), grid, block)
+        if not sync:
+            return state
+        s.synchronize()
+        return state["y"], int(state["err"][0].item())
+
     def pin(self, path, flags=0) -> int:
         """Open `path` and keep it open across launches (later gopen calls need no RPC)."""
         return self.fileop(path, "pin", flags=flags)

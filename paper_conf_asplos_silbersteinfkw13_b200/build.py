@@ -10,7 +10,7 @@ ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
 INC = os.path.join(ROOT, "include")
 LIB = os.path.join(PKG, "libgpufs.so")
-SOURCES = [os.path.join(CSRC, f) for f in ("gfs_kernels.cu", "gfs_grep.cu", "gfs_host.cpp")]
+SOURCES = [os.path.join(CSRC, f) for f in ("gfs_kernels.cu", "gfs_grep.cu", "gfs_matvec.cu", "gfs_host.cpp")]
 HEADERS = [os.path.join(INC, f) for f in ("gpufs.h", "gpufs_layout.h", "gpufs_device.cuh")]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]

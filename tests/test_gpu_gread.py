@@ -113,8 +113,8 @@ def test_locked_traversal_same_bytes(g, shmdir, locked):
         check_calls(path, size, offs, lens, ret, dst, dstoff)
     except AssertionError as e:
         raise AssertionError(f"{e} | dev {st} | host {hs} | info {info}")
-    if locked:
-        assert st["locked"] > 0 and st["lockfree"] == 0
+    if locked:  # every first lookup takes the lock (busy retries may go lock-free)
+        assert st["locked"] >= 300
     else:
         assert st["lockfree"] > 0
 
