@@ -241,6 +241,9 @@ def run_ours(args):
     grep = None
     if not args.no_grep:
         grep = grep_phase(args, torch, g, gen, dev, stream, hbm, rank, ws, local, dist)
+    mv = None
+    if not args.no_matvec:
+        mv = matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local)
 
     tmax = torch.tensor([ms], device=dev)
     if ws > 1:
@@ -278,6 +281,8 @@ def run_ours(args):
         line["hit"] = hit
     if grep:
         line["grep"] = grep
+    if mv:
+        line["matvec"] = mv
     if not args.no_cpu:
         line["cpu_baseline"] = cpu_baseline(args, path, size)
     print(json.dumps(line), flush=True)
@@ -417,6 +422,54 @@ def grep_phase(args, torch, g, gen, dev, stream, hbm, rank, ws, local, dist):
     return res
 
 
+def matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local):
+    """C3 (configs[2]): y = A x, A (rows x 131072 fp32) larger than the 2 GiB cache,
+    read through gmmap, y through gwrite + gfsync."""
+    import oracle
+    rows, cols = args.mv_rows, 131072
+    m = gen.matrix_files(f"/dev/shm/gfs_bench_c3_r{rank}", rows, cols, seed=3 + rank)
+    ypath = f"/dev/shm/gfs_bench_c3_r{rank}/y.f32"
+    nbytes = rows * cols * 4
+    with g.GpuFS(cache_bytes=2 << 30, page_size=2 << 20, device=local, daemon_threads=args.daemon_threads,
+                 max_batch=1, timeout_ms=args.timeout_ms) as fs:
+        state = None
+        ts = []
+        for it in range(3):
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            with torch.cuda.stream(stream):
+                e0.record(stream)
+                state = fs.matvec(m["A"], m["x"], ypath, rows, cols, stream=stream, sync=False, state=state)
+                e1.record(stream)
+                stream.synchronize()
+            ts.append(e0.elapsed_time(e1))
+        err = int(state["err"][0].item())
+        y = state["y"].cpu().numpy().astype(np.float64)
+        st = fs.stats()
+    ms = float(np.median(ts))
+    gbs = nbytes / (ms * 1e-3) / 1e9
+    rng = np.random.default_rng(0)
+    sample = np.unique(np.concatenate([np.arange(8), rng.integers(0, rows, size=56)]))
+    ref = np.array([oracle.matvec(m["A"], m["x"], rows, cols, row0=int(r), nrows=1)[0] for r in sample])
+    relerr = float(np.max(np.abs(y[sample] - ref) / np.abs(ref)))
+    yh = np.fromfile(ypath, dtype="<f4").astype(np.float64)
+    out = {"workload": f"C3: {rows} x {cols} fp32 matrix ({nbytes >> 20} MiB) > 2 GiB cache, 2 MiB pages, "
+                       f"gmmap rows, gwrite+gfsync y",
+           "GBps": round(gbs, 3), "ms": round(ms, 3), "err": err,
+           "roofline": {"bound": "h2d", "achieved": round(gbs, 3), "peak": round(h2d, 3), "unit": "GB/s",
+                        "frac": round(gbs / h2d, 4)},
+           "max_rel_err_sampled_rows": relerr, "parity_ok": relerr <= 1e-5 and np.array_equal(yh, y),
+           "misses": st["miss"], "evictions": st["evict"]}
+    if not args.no_cpu:
+        t0 = time.perf_counter()
+        n = min(rows, 2048)
+        oracle.matvec(m["A"], m["x"], rows, cols, row0=0, nrows=n, nthreads=os.cpu_count() or 1)
+        dt = time.perf_counter() - t0
+        out["cpu_baseline"] = {"value": round(n * cols * 4 / dt / 1e9, 3), "unit": "GB/s",
+                               "cores": os.cpu_count(), "kind": "oracle",
+                               "sample": f"first {n} rows, float64, nproc threads"}
+    return out
+
+
 def cpu_baseline(args, path, size):
     import oracle
     sample = min(size, args.ref_sample_mib << 20)
@@ -447,6 +500,8 @@ def main():
     ap.add_argument("--timeout-ms", type=int, default=60000)
     ap.add_argument("--no-hit", action="store_true")
     ap.add_argument("--no-grep", action="store_true")
+    ap.add_argument("--no-matvec", action="store_true")
+    ap.add_argument("--mv-rows", type=int, default=11200)  # 5.6 GB (Fig. 8's 5600 MB point x2)
     ap.add_argument("--grep-files", type=int, default=30000)
     ap.add_argument("--grep-mib", type=int, default=500)
     ap.add_argument("--grep-cache-gib", type=int, default=4)
