@@ -54,6 +54,7 @@ namespace detail {
 namespace {  // internal linkage: the header is included by several translation units
 
 constexpr int kBusy = -10000;  // lookup result: page being filled/evicted elsewhere
+constexpr int kLeafCache = 32; // per-block leaf-node cache entries
 
 // ------------------------------------------------------------------ PTX
 __device__ __forceinline__ uint64_t now_ns() {
@@ -199,6 +200,17 @@ struct Scratch {
   uint64_t cached_grid;
   uint32_t cached_blk;
   int32_t cached_fd;
+  // Leaf-node ids of the cached file's radix tree, direct-mapped by page >> 8:
+  // interior nodes never change while the file is open, so a block that holds
+  // it skips the upper levels of the walk (one dependent L2 load fewer).
+  // Entries are ((page >> 8) + 1) << 32 | node, one 64-bit store each.
+  uint64_t leaf[kLeafCache];
+  uint32_t lc_ok;  // this call's snapshot is the cached one (leaf cache usable)
+  // mbarrier for TMA bulk copies into shared memory (same validity key)
+  uint64_t mbar;
+  uint64_t mbar_grid;
+  uint32_t mbar_blk;
+  uint32_t mbar_phase;
   int32_t frame[GFS_MAX_BATCH];   // >= 0 held frame; kBusy / -errno otherwise
   int32_t stage[GFS_MAX_BATCH];   // staging slot to pull from (>= 0), or -1
   uint32_t fill[GFS_MAX_BATCH];   // 1: this block installed the frame and must fill it
@@ -513,6 +525,35 @@ __device__ __forceinline__ void block_zero(uint8_t* dst, uint64_t n, int tid, in
   for (uint64_t k = head + (nv << 4) + tid; k < n; k += nthr) dst[k] = 0;
 }
 
+// ------------------------------------------------------------------ TMA bulk copy
+// cp.async.bulk global -> shared, completion counted in bytes on an mbarrier
+// (SASS UBLKCP). Used by gread when the destination is shared memory: one
+// thread moves the whole span, the data never passes through registers.
+__device__ __forceinline__ uint32_t smem_u32(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
+__device__ __forceinline__ void mbar_init(uint64_t* m) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(smem_u32(m)) : "memory");
+  asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+}
+__device__ __forceinline__ void mbar_expect_tx(uint64_t* m, uint32_t bytes) {
+  asm volatile("{ .reg .b64 st; mbarrier.arrive.expect_tx.shared::cta.b64 st, [%0], %1; }" ::"r"(smem_u32(m)),
+               "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void tma_load(void* dst_smem, const void* src, uint32_t bytes, uint64_t* m) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                   smem_u32(dst_smem)),
+               "l"(src), "r"(bytes), "r"(smem_u32(m))
+               : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* m, uint32_t phase) {
+  asm volatile(
+      "{ .reg .pred P1;\n"
+      "WAIT_%=: mbarrier.try_wait.parity.shared::cta.b64 P1, [%0], %1;\n"
+      "@!P1 bra WAIT_%=;\n}" ::"r"(smem_u32(m)),
+      "r"(phase)
+      : "memory");
+}
+
 // ------------------------------------------------------------------ frames
 __device__ __forceinline__ uint8_t* frame_ptr(const gfs_ctx* c, uint32_t f) {
   return c->pool + ((size_t)f << c->page_shift);
@@ -658,11 +699,22 @@ __device__ __forceinline__ void frame_abandon(const gfs_ctx* c, uint32_t f) {
 // tag the evictor has since replaced). All accesses are strong gpu-scope
 // operations served at L2, so no L1 line can be stale. Returns the frame, or
 // -1 to take the full (acquire/release) path.
-__device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
+__device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs, uint64_t page,
+                                           uint64_t* leaf_cache = nullptr) {
   uint32_t node = fs.root;
-  for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
-    node = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
-    if (!node) return -1;
+  if (fs.height > 1) {
+    const uint32_t key = (uint32_t)(page >> GFS_FANOUT_SHIFT);
+    const uint64_t ent = leaf_cache ? leaf_cache[key & (kLeafCache - 1)] : 0;
+    if (ent >> 32 == (uint64_t)key + 1) {
+      node = (uint32_t)ent;
+    } else {
+      for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
+        node = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT +
+                      ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
+        if (!node) return -1;
+      }
+      if (leaf_cache) leaf_cache[key & (kLeafCache - 1)] = (((uint64_t)key + 1) << 32) | node;
+    }
   }
   const uint32_t s = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
   if (!s) return -1;
@@ -740,6 +792,7 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     }
     const uint32_t s = ld_acq(slot);
     bool done = false;
+    int pinned = -1;  // stale frame kept referenced across the install CAS
     if (s) {
       const uint32_t f = s - 1;
       const uint32_t old = atom_add_acq(&c->f_state[f], 1u);
@@ -749,17 +802,16 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
           ctr(c, GFS_C_HIT);
           out.frame = (int)f;
           done = true;
-        } else {
+        } else if (old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
           atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
-          if (old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
-            ctr(c, GFS_C_BUSY);
-            out.frame = kBusy;
-            done = true;
-          }
-          // ERROR with no fill in flight: stale, install over it
+          ctr(c, GFS_C_BUSY);
+          out.frame = kBusy;
+          done = true;
+        } else {
+          atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);  // ERROR, no fill in flight: stale, install over it
         }
       } else {
-        atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+        atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);  // stale slot: install over it
       }
       if (!done) {
         ++attempt;
@@ -771,10 +823,22 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     // miss (or stale slot): install a new frame for `want`
     const int g = alloc_frame(c, want, fs.fdx);
     if (g < 0) {
+      if (pinned >= 0) atom_add_rel(&c->f_state[pinned], 0xFFFFFFFFu);
       out.frame = g;
       break;
     }
-    if (atom_cas(slot, s, (uint32_t)g + 1u) != s) {
+    bool won = atom_cas(slot, s, (uint32_t)g + 1u) == s;
+    if (pinned >= 0) atom_add_rel(&c->f_state[pinned], 0xFFFFFFFFu);
+    if (won && s && (s - 1) != (uint32_t)g && ld_acq64(&c->f_tag[s - 1]) == want) {
+      // ABA: between our read of the stale value F+1 and our CAS, F was
+      // evicted and installed again for this very page (same slot value), and
+      // may already hold written data. Put it back and retry: otherwise F
+      // would be orphaned with its dirty bytes. (Nobody else can have replaced
+      // our unpublished frame meanwhile: it is FILLING with this tag, BUSY.)
+      atom_cas(slot, (uint32_t)g + 1u, s);
+      won = false;
+    }
+    if (!won) {
       frame_abandon(c, (uint32_t)g);
       ++attempt;
       ctr(c, GFS_C_RETRY);
@@ -838,7 +902,7 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
         // Retries of busy pages always try the lock-free path first: in the
         // locked ablation, hundreds of lanes re-taking the file lock while
         // they wait starve the lanes that still have to install pages.
-        int f = (fast || round > 0) ? lookup_fast(c, fs, pb + tid) : -1;
+        int f = (fast || round > 0) ? lookup_fast(c, fs, pb + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
         if (f < 0 && round > 0 && peek_busy(c, fs, pb + tid)) {
           // still being filled/evicted elsewhere: look again later without
           // taking the lock (lock-taking retries starve the installers)
@@ -1249,6 +1313,13 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
       sc.cached_grid = detail::grid_id();
       sc.cached_blk = detail::block_linear();
       sc.cached_fd = fd;
+      for (int i = 0; i < detail::kLeafCache; ++i) sc.leaf[i] = 0;
+    }
+    if (sc.mbar_grid != detail::grid_id() || sc.mbar_blk != detail::block_linear()) {
+      detail::mbar_init(&sc.mbar);  // first gopen of this block in this launch
+      sc.mbar_phase = 0;
+      sc.mbar_grid = detail::grid_id();
+      sc.mbar_blk = detail::block_linear();
     }
   }
   __syncthreads();
@@ -1308,10 +1379,13 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   if (tid < 32) {
     if (tid == 0) {
       FileSnap s;
-      if (!snap_fd_cached(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
+      const bool cached = sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id();
+      if (cached) s = sc.cached;
+      if (!(cached || snap_fd(c, fd, &s)) || (s.oflags & GFS_O_GWRONCE)) {
         sc.ret = -EBADF;
       } else {
         sc.fs = s;
+        sc.lc_ok = cached ? 1u : 0u;
         sc.ret = off >= s.size ? 0 : (int64_t)(len < s.size - off ? len : s.size - off);
         ctr(c, GFS_C_GREAD_CALLS);
         if (sc.ret > 0) ctr(c, GFS_C_GREAD_BYTES, (unsigned long long)sc.ret);
@@ -1324,7 +1398,7 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
       const uint32_t cnt = (uint32_t)((q1 - q0 + 1) < B ? (q1 - q0 + 1) : B);
       if (tid < (int)cnt) {
         const FileSnap fs0 = sc.fs;
-        int f = fast ? lookup_fast(c, fs0, q0 + tid) : -1;
+        int f = fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
         if (f < 0) {
           const Lk r = lookup_try(c, fs0, q0 + tid);
           sc.frame[tid] = r.frame;
@@ -1344,18 +1418,43 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   if (n <= 0) return n;
   const FileSnap fs = sc.fs;
   const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
+  // TMA path: shared-memory destination, everything 16-byte aligned, the
+  // block's mbarrier initialised in this launch (set up by its gopen).
+  const bool tma = __isShared(dst) && ((((uintptr_t)dst) | off | (uint64_t)n) & 15) == 0 &&
+                   sc.mbar_grid == grid_id() && sc.mbar_blk == block_linear();
   for (uint64_t pb = p0; pb <= p1; pb += B) {
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
     const int err = acquire_batch(c, sc, fs, pb, cnt, pb == p0);
     if (err) return err;
-    for (uint32_t i = 0; i < cnt; ++i) {
-      const uint64_t p = pb + i;
-      const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
-      const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-      block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
-                            e - s, tid, nthr);
+    const uint64_t bs = pb == p0 ? (off & (P - 1)) : 0;
+    const uint64_t be = pb + cnt - 1 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+    const uint64_t batch_bytes = ((uint64_t)cnt << shift) - bs - (P - be);
+    if (tma && batch_bytes < (1u << 20)) {  // mbarrier tx-count limit
+      const uint32_t ph = sc.mbar_phase;
+      if (tid == 0) {
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
+        mbar_expect_tx(&sc.mbar, (uint32_t)batch_bytes);
+        for (uint32_t i = 0; i < cnt; ++i) {
+          const uint64_t p = pb + i;
+          const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+          const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+          tma_load((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+                   (uint32_t)(e - s), &sc.mbar);
+        }
+      }
+      mbar_wait(&sc.mbar, ph);
+      __syncthreads();
+      if (tid == 0) sc.mbar_phase = ph ^ 1u;
+    } else {
+      for (uint32_t i = 0; i < cnt; ++i) {
+        const uint64_t p = pb + i;
+        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+        block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+                              e - s, tid, nthr);
+      }
+      __syncthreads();
     }
-    __syncthreads();
     if (tid < (int)cnt) frame_release(c, (uint32_t)sc.frame[tid]);
   }
   return n;
@@ -1378,6 +1477,7 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
       sc.ret = -EINVAL;
     } else {
       sc.fs = s;
+      sc.lc_ok = 0;
       sc.ret = (int64_t)len;
       ctr(c, GFS_C_GWRITE_CALLS);
     }
@@ -1525,6 +1625,7 @@ __device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int pr
       sc.aux = -EBADF;
     } else if (off < s.size && len > 0) {
       sc.fs = s;
+      sc.lc_ok = (sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id()) ? 1u : 0u;
       sc.ret = 1;
     }
   }

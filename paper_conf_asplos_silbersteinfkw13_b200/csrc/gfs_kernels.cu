@@ -182,12 +182,26 @@ __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const cha
   }
   uint64_t s = 0;
   const uint64_t* my = offs + (size_t)blockIdx.x * calls;
+  // raw baseline: the same copy without GPUfs — TMA bulk copy like gread's
+  // shared-memory path, so the comparison isolates the cache's cost
+  __shared__ uint64_t raw_mbar;
+  if (raw) {
+    if (tid == 0) detail::mbar_init(&raw_mbar);
+    __syncthreads();
+  }
+  uint32_t ph = 0;
   for (uint32_t i = 0; i < calls; ++i) {
     const uint64_t o = my[i];
     int64_t r;
     if (raw) {
       __syncthreads();
-      detail::block_copy_from_frame(smem, rawp + o, chunk, tid, nthr);
+      if (tid == 0) {
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        detail::mbar_expect_tx(&raw_mbar, chunk);
+        detail::tma_load(smem, rawp + o, chunk, &raw_mbar);
+      }
+      detail::mbar_wait(&raw_mbar, ph);
+      ph ^= 1u;
       __syncthreads();
       r = chunk;
     } else {

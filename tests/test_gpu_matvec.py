@@ -44,3 +44,20 @@ def test_matvec_vs_oracle(g, shmdir, rows, cols, P, cache_mb, integer):
         assert np.max(np.abs(yd - ref) / np.abs(ref)) <= 1e-5
     if rows * cols * 4 > (cache_mb << 20):
         assert st["evict"] > 0
+
+
+def test_concurrent_row_writes_under_eviction(g, shmdir):
+    """Regression: 40 blocks gwrite 4-byte rows into one y page while the matrix
+    stream evicts it again and again (4-frame cache). An ABA in the install CAS
+    used to orphan a live dirty frame and lose rows on the host."""
+    rows, cols = 40, 131072
+    m = gen.matrix_files(shmdir, rows, cols, seed=3, integer=True)
+    ref = oracle.matvec(m["A"], m["x"], rows, cols, nthreads=4).astype(np.float32)
+    for it in range(6):
+        ypath = os.path.join(shmdir, f"y{it}.f32")
+        with g.GpuFS(cache_bytes=8 << 20, page_size=1 << 21, timeout_ms=60000, daemon_threads=4,
+                     max_batch=1) as fs:
+            y, err = fs.matvec(m["A"], m["x"], ypath, rows, cols, grid=40)
+        assert err == 0
+        assert np.array_equal(y.cpu().numpy(), ref)
+        assert np.array_equal(np.fromfile(ypath, dtype="<f4"), ref), it
