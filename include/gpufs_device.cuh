@@ -153,6 +153,53 @@ __device__ __forceinline__ unsigned long long atom_add64(unsigned long long* p, 
   asm volatile("atom.relaxed.gpu.global.add.u64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
   return r;
 }
+// 64-bit frame-state / tree-slot atomics (generation << 32 | low word)
+__device__ __forceinline__ uint64_t a64_add_rlx(uint64_t* p, uint64_t v) {
+  uint64_t r;
+  asm volatile("atom.relaxed.gpu.global.add.u64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint64_t a64_add_acq(uint64_t* p, uint64_t v) {
+  uint64_t r;
+  asm volatile("atom.acquire.gpu.global.add.u64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint64_t a64_add_rel(uint64_t* p, uint64_t v) {
+  uint64_t r;
+  asm volatile("atom.release.gpu.global.add.u64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ void r64_add_rlx(uint64_t* p, uint64_t v) {
+  asm volatile("red.relaxed.gpu.global.add.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ uint64_t a64_and_rel(uint64_t* p, uint64_t v) {
+  uint64_t r;
+  asm volatile("atom.release.gpu.global.and.b64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint64_t a64_or_rel(uint64_t* p, uint64_t v) {
+  uint64_t r;
+  asm volatile("atom.release.gpu.global.or.b64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint64_t a64_cas(uint64_t* p, uint64_t cmp, uint64_t val) {
+  uint64_t r;
+  asm volatile("atom.acq_rel.gpu.global.cas.b64 %0, [%1], %2, %3;"
+               : "=l"(r) : "l"(p), "l"(cmp), "l"(val) : "memory");
+  return r;
+}
+constexpr uint64_t kRefDec = ~0ull;  // ref - 1 (never borrows: the ref being dropped is >= 1)
+__device__ __forceinline__ uint64_t fl64(uint32_t flags) { return ~(uint64_t)flags; }  // and-mask clearing flags
+// Leaf slot value for frame f of generation gen.
+__device__ __forceinline__ uint64_t slot_val(uint32_t f, uint32_t gen) { return ((uint64_t)gen << 32) | (f + 1u); }
+// Claim frame f for exclusive use (EVICTING) if its low word is exactly `low`
+// (0: unreferenced, no flags). Keeps the generation.
+__device__ __forceinline__ bool claim_frame(uint64_t* st, uint32_t low) {
+  const uint64_t v = ld_rlx64(st);
+  if ((uint32_t)v != low) return false;
+  return a64_cas(st, v, (v & 0xFFFFFFFF00000000ull) | GFS_ST_EVICTING) == v;
+}
+
 __device__ __forceinline__ void backoff(uint32_t& ns) {
   __nanosleep(ns);
   ns = ns < 4096 ? ns * 2 : 4096;
@@ -211,6 +258,7 @@ struct Scratch {
   uint64_t mbar_grid;
   uint32_t mbar_blk;
   uint32_t mbar_phase;
+  uint32_t quick;  // this gread's one-page TMA copy was issued by lane 0 before the barrier
   int32_t frame[GFS_MAX_BATCH];   // >= 0 held frame; kBusy / -errno otherwise
   int32_t stage[GFS_MAX_BATCH];   // staging slot to pull from (>= 0), or -1
   uint32_t fill[GFS_MAX_BATCH];   // 1: this block installed the frame and must fill it
@@ -369,7 +417,7 @@ __device__ uint32_t node_alloc(const gfs_ctx* c) {
 
 __device__ void node_free_one(const gfs_ctx* c, uint32_t n) {
   uint4* p = (uint4*)(c->nodes + (size_t)n * GFS_FANOUT);
-  for (int i = 0; i < (int)(GFS_FANOUT / 4); ++i) p[i] = make_uint4(0, 0, 0, 0);
+  for (int i = 0; i < (int)(GFS_FANOUT / 2); ++i) p[i] = make_uint4(0, 0, 0, 0);
   __threadfence();
   spin_lock(c->node_lock);
   uint32_t top = *(volatile uint32_t*)c->node_free_top;
@@ -391,7 +439,7 @@ __device__ void tree_free(const gfs_ctx* c, uint32_t root, uint32_t height) {
     const uint32_t h = height - (uint32_t)sp;
     if (h > 1 && stk_idx[sp] < GFS_FANOUT) {
       const uint32_t i = stk_idx[sp]++;
-      const uint32_t ch = c->nodes[(size_t)node * GFS_FANOUT + i];
+      const uint32_t ch = (uint32_t)c->nodes[(size_t)node * GFS_FANOUT + i];
       if (ch) {
         ++sp;
         stk_node[sp] = ch;
@@ -405,15 +453,15 @@ __device__ void tree_free(const gfs_ctx* c, uint32_t root, uint32_t height) {
 }
 
 // Walk (creating interior nodes if `create`) to the leaf slot of `page`.
-// Interior entries hold child node ids; leaf entries hold frame id + 1.
+// Interior entries hold child node ids; leaf entries hold slot_val(frame, gen).
 // New nodes are zeroed before the publishing CAS.
-__device__ uint32_t* walk(const gfs_ctx* c, uint32_t root, uint32_t height, uint64_t page, bool create,
+__device__ uint64_t* walk(const gfs_ctx* c, uint32_t root, uint32_t height, uint64_t page, bool create,
                           int* err) {
   uint32_t node = root;
   for (int lvl = (int)height - 1; lvl >= 1; --lvl) {
     const uint32_t idx = (uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & (GFS_FANOUT - 1);
-    uint32_t* sp = c->nodes + (size_t)node * GFS_FANOUT + idx;
-    uint32_t ch = ld_acq(sp);
+    uint64_t* sp = c->nodes + (size_t)node * GFS_FANOUT + idx;
+    uint32_t ch = (uint32_t)ld_acq64(sp);
     if (!ch) {
       if (!create) return nullptr;
       const uint32_t n = node_alloc(c);
@@ -422,7 +470,7 @@ __device__ uint32_t* walk(const gfs_ctx* c, uint32_t root, uint32_t height, uint
         return nullptr;
       }
       __threadfence();
-      const uint32_t prev = atom_cas(sp, 0u, n);
+      const uint32_t prev = (uint32_t)a64_cas(sp, 0ull, n);
       if (prev) {
         node_free_one(c, n);
         ch = prev;
@@ -559,7 +607,8 @@ __device__ __forceinline__ uint8_t* frame_ptr(const gfs_ctx* c, uint32_t f) {
   return c->pool + ((size_t)f << c->page_shift);
 }
 
-__device__ __forceinline__ void frame_init(const gfs_ctx* c, uint32_t f, uint64_t tag, uint32_t fdx) {
+// Returns the frame's new generation (the value its tree slot must carry).
+__device__ __forceinline__ uint32_t frame_init(const gfs_ctx* c, uint32_t f, uint64_t tag, uint32_t fdx) {
   st_rlx64(&c->f_tag[f], tag);
   st_rlx(&c->f_file[f], fdx);
   st_rlx(&c->f_valid[f], 0);
@@ -567,10 +616,11 @@ __device__ __forceinline__ void frame_init(const gfs_ctx* c, uint32_t f, uint64_
   st_rlx(&c->f_hi[f], 0);
   st_rlx(&c->f_written[f], 0);
   st_rlx(&c->f_stamp[f], stamp_now());
-  // EVICTING -> FILLING|1 as an atomic delta: readers that found the frame
-  // through a stale slot may hold transient +1s they are about to undo, so the
-  // state word is never overwritten with a plain store.
-  atom_add_rel(&c->f_state[f], GFS_ST_FILLING + 1u - GFS_ST_EVICTING);
+  // EVICTING -> FILLING|1 and generation + 1 as one atomic delta: readers that
+  // found the frame through a stale slot may hold transient +1s they are about
+  // to undo, so the state word is never overwritten with a plain store.
+  const uint64_t delta = (1ull << 32) + (uint64_t)GFS_ST_FILLING + 1ull - (uint64_t)GFS_ST_EVICTING;
+  return (uint32_t)((a64_add_rel(&c->f_state[f], delta) + delta) >> 32);
 }
 
 // Write back a frame's dirty range from one thread (the caller owns the frame:
@@ -616,13 +666,14 @@ __device__ __forceinline__ uint32_t frame_tier(const gfs_ctx* c, uint32_t f, uin
 // Allocate a frame for `tag`: never-used frames first, else evict the oldest
 // reclaimable frame of a 32-frame window (sampled LRU, tiered by P:L651-657),
 // writing back a dirty victim first. Runs in the calling thread.
-// Returns the frame in state FILLING|1 with its tag set, or -ENOMEM.
-__device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx) {
+// Returns the frame in state FILLING|1 with its tag set (and its new
+// generation in *gen), or -ENOMEM.
+__device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx, uint32_t* gen) {
   const uint32_t N = c->nframes;
   if (ld_rlx(c->fresh_next) < N) {
     const uint32_t f = atomicAdd(c->fresh_next, 1u);
     if (f < N) {
-      frame_init(c, f, tag, fdx);
+      *gen = frame_init(c, f, tag, fdx);
       return (int)f;
     }
   }
@@ -633,31 +684,32 @@ __device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx) {
     const uint32_t w = atomicAdd(c->hand, 32u);
     int best = -1;
     uint64_t best_key = ~0ull;
-    uint32_t best_st = 0;
+    uint64_t best_st = 0;
 #pragma unroll 4
     for (uint32_t j = 0; j < 32; ++j) {
       const uint32_t f = (uint32_t)(((uint64_t)w + j) % N);
-      const uint32_t st = ld_rlx(&c->f_state[f]);
-      if (st & ~GFS_ST_ERROR) continue;  // referenced, filling or being evicted
-      const uint64_t key = ((uint64_t)frame_tier(c, f, st) << 32) | ld_rlx(&c->f_stamp[f]);
+      const uint64_t st = ld_rlx64(&c->f_state[f]);
+      if ((uint32_t)st & ~GFS_ST_ERROR) continue;  // referenced, filling or being evicted
+      const uint64_t key = ((uint64_t)frame_tier(c, f, (uint32_t)st) << 32) | ld_rlx(&c->f_stamp[f]);
       if (key < best_key) {
         best_key = key;
         best = (int)f;
         best_st = st;
       }
     }
-    if (best >= 0 && atom_cas(&c->f_state[best], best_st, GFS_ST_EVICTING) == best_st) {
+    if (best >= 0 &&
+        a64_cas(&c->f_state[best], best_st, (best_st & 0xFFFFFFFF00000000ull) | GFS_ST_EVICTING) == best_st) {
       const uint32_t f = (uint32_t)best;
       if (ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) {
         const uint32_t fi = ld_rlx(&c->f_file[f]);
         const int32_t r = frame_writeback_lane(c, f, ld_rlx(&c->files[fi].hfid));
         if (r < 0) {  // keep the dirty page, try another victim
-          atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+          a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
           continue;
         }
       }
       ctr(c, GFS_C_EVICT);
-      frame_init(c, f, tag, fdx);
+      *gen = frame_init(c, f, tag, fdx);
       return (int)f;
     }
     if (round > 0 && round % windows == 0) {
@@ -675,28 +727,40 @@ __device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx) {
 // otherwise), so a relaxed decrement suffices.
 __device__ __forceinline__ void frame_release(const gfs_ctx* c, uint32_t f) {
   st_rlx(&c->f_stamp[f], stamp_now());
-  red_add_rlx(&c->f_state[f], 0xFFFFFFFFu);  // ref - 1
+  r64_add_rlx(&c->f_state[f], kRefDec);  // ref - 1
 }
 // Release after writing a frame (gwrite): the dirty-range updates must be
 // visible before the reference drops (gfsync only syncs unreferenced frames).
 __device__ __forceinline__ void frame_release_rel(const gfs_ctx* c, uint32_t f) {
   st_rlx(&c->f_stamp[f], stamp_now());
-  atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+  a64_add_rel(&c->f_state[f], kRefDec);
+}
+
+// Drop the page a published frame holds: tag cleared, generation + 1 (every
+// tree slot naming the old generation is now stale), `flag` (held by the
+// caller) cleared, in one atomic delta.
+__device__ __forceinline__ void frame_retire(const gfs_ctx* c, uint32_t f, uint32_t flag) {
+  st_rlx64(&c->f_tag[f], GFS_TAG_NONE);
+  a64_add_rel(&c->f_state[f], (1ull << 32) - (uint64_t)flag);
 }
 
 // Give back a frame we installed but could not publish (lost the CAS race).
 __device__ __forceinline__ void frame_abandon(const gfs_ctx* c, uint32_t f) {
   st_rel64(&c->f_tag[f], GFS_TAG_NONE);
-  atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
-  atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+  a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));
+  a64_add_rel(&c->f_state[f], kRefDec);
 }
 
 // ------------------------------------------------------------------ page lookup
 // Cache-hit fast path (one optimistic attempt): relaxed walk
-// without creating nodes, relaxed incref, then the tag load made
-// address-dependent on the incref's result so it cannot be performed before
-// it (a plain relaxed load could be satisfied first and validate against a
-// tag the evictor has since replaced). All accesses are strong gpu-scope
+// without creating nodes, then ONE relaxed atomic increment of the frame's
+// state word that both takes the reference and validates the slot: the
+// generation it returns must equal the one stored in the slot (the frame was
+// not reassigned since it was installed for this page) and no FILLING /
+// EVICTING / ERROR flag may be set. This replaces the paper's tag re-check
+// by a per-frame generation, so a hit costs two dependent L2
+// round trips instead of three. The tree cannot be freed under us: the
+// caller's block holds the file open. All accesses are strong gpu-scope
 // operations served at L2, so no L1 line can be stale. Returns the frame, or
 // -1 to take the full (acquire/release) path.
 __device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs, uint64_t page,
@@ -709,27 +773,23 @@ __device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs,
       node = (uint32_t)ent;
     } else {
       for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
-        node = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT +
-                      ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
+        node = (uint32_t)ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT +
+                                  ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
         if (!node) return -1;
       }
       if (leaf_cache) leaf_cache[key & (kLeafCache - 1)] = (((uint64_t)key + 1) << 32) | node;
     }
   }
-  const uint32_t s = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
-  if (!s) return -1;
-  const uint32_t f = s - 1;
-  const uint32_t old = atom_add_rlx(&c->f_state[f], 1u);
-  // bit 30 of the state word is never set, so fdep == f; the dependency is real
-  const uint32_t fdep = min(f, f + (old & 0x40000000u));
-  const uint64_t tag = ld_rlx64(&c->f_tag[fdep]);
-  if (tag == (((uint64_t)fs.uid << 32) | (uint32_t)page) &&
-      !(old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
+  const uint64_t s = ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
+  if (!(uint32_t)s) return -1;
+  const uint32_t f = (uint32_t)s - 1u;
+  const uint64_t old = a64_add_rlx(&c->f_state[f], 1ull);
+  if ((old >> 32) == (s >> 32) && !((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
     ctr(c, GFS_C_HIT);
     ctr(c, GFS_C_LOCKFREE);
     return (int)f;
   }
-  red_add_rlx(&c->f_state[f], 0xFFFFFFFFu);
+  r64_add_rlx(&c->f_state[f], kRefDec);
   return -1;
 }
 
@@ -738,15 +798,14 @@ __device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs,
 __device__ __forceinline__ bool peek_busy(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
   uint32_t node = fs.root;
   for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
-    node = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
+    node = (uint32_t)ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT +
+                              ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
     if (!node) return false;
   }
-  const uint32_t s = ld_rlx(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
-  if (!s) return false;
-  const uint32_t f = s - 1;
-  const uint32_t st = ld_rlx(&c->f_state[f]);
-  return (st & (GFS_ST_FILLING | GFS_ST_EVICTING)) &&
-         ld_rlx64(&c->f_tag[f]) == (((uint64_t)fs.uid << 32) | (uint32_t)page);
+  const uint64_t s = ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
+  if (!(uint32_t)s) return false;
+  const uint64_t st = ld_rlx64(&c->f_state[(uint32_t)s - 1u]);
+  return (st >> 32) == (s >> 32) && ((uint32_t)st & (GFS_ST_FILLING | GFS_ST_EVICTING));
 }
 
 struct Lk {
@@ -772,7 +831,7 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
   const bool always_lock = (c->flags & GFS_F_LOCKED_TRAVERSAL) != 0;  // K5 ablation
   bool used_lock = false;
   int attempt = 0;
-  uint32_t* slot = nullptr;
+  uint64_t* slot = nullptr;
   for (;;) {
     // The lock (when taken) covers the traversal only: walk, slot read,
     // reference + validation. Fills and RPCs run unlocked.
@@ -790,28 +849,28 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
         break;
       }
     }
-    const uint32_t s = ld_acq(slot);
+    const uint64_t s = ld_acq64(slot);
     bool done = false;
-    int pinned = -1;  // stale frame kept referenced across the install CAS
-    if (s) {
-      const uint32_t f = s - 1;
-      const uint32_t old = atom_add_acq(&c->f_state[f], 1u);
-      const uint64_t tag = ld_acq64(&c->f_tag[f]);
-      if (tag == want) {
-        if (!(old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
+    if ((uint32_t)s) {
+      const uint32_t f = (uint32_t)s - 1u;
+      const uint64_t old = a64_add_acq(&c->f_state[f], 1ull);
+      // same generation as the slot <=> the frame still holds this page (the
+      // tag check is kept as a belt-and-braces test on the slow path)
+      if ((old >> 32) == (s >> 32) && ld_acq64(&c->f_tag[f]) == want) {
+        if (!((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
           ctr(c, GFS_C_HIT);
           out.frame = (int)f;
           done = true;
-        } else if (old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
-          atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);
+        } else if ((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
+          a64_add_rel(&c->f_state[f], kRefDec);
           ctr(c, GFS_C_BUSY);
           out.frame = kBusy;
           done = true;
         } else {
-          atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);  // ERROR, no fill in flight: stale, install over it
+          a64_add_rel(&c->f_state[f], kRefDec);  // ERROR, no fill in flight: stale, install over it
         }
       } else {
-        atom_add_rel(&c->f_state[f], 0xFFFFFFFFu);  // stale slot: install over it
+        a64_add_rel(&c->f_state[f], kRefDec);  // stale slot: install over it
       }
       if (!done) {
         ++attempt;
@@ -820,24 +879,16 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     }
     if (lk) spin_unlock(lockp);
     if (done) break;
-    // miss (or stale slot): install a new frame for `want`
-    const int g = alloc_frame(c, want, fs.fdx);
+    // miss (or stale slot): install a new frame for `want`. The slot value
+    // carries the frame's generation, so the CAS cannot succeed against a
+    // value that was replaced and restored in between (no ABA).
+    uint32_t gen = 0;
+    const int g = alloc_frame(c, want, fs.fdx, &gen);
     if (g < 0) {
-      if (pinned >= 0) atom_add_rel(&c->f_state[pinned], 0xFFFFFFFFu);
       out.frame = g;
       break;
     }
-    bool won = atom_cas(slot, s, (uint32_t)g + 1u) == s;
-    if (pinned >= 0) atom_add_rel(&c->f_state[pinned], 0xFFFFFFFFu);
-    if (won && s && (s - 1) != (uint32_t)g && ld_acq64(&c->f_tag[s - 1]) == want) {
-      // ABA: between our read of the stale value F+1 and our CAS, F was
-      // evicted and installed again for this very page (same slot value), and
-      // may already hold written data. Put it back and retry: otherwise F
-      // would be orphaned with its dirty bytes. (Nobody else can have replaced
-      // our unpublished frame meanwhile: it is FILLING with this tag, BUSY.)
-      atom_cas(slot, (uint32_t)g + 1u, s);
-      won = false;
-    }
+    const bool won = a64_cas(slot, s, slot_val((uint32_t)g, gen)) == s;
     if (!won) {
       frame_abandon(c, (uint32_t)g);
       ++attempt;
@@ -859,9 +910,9 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     if (nb && st >= 0) r = rpc_call(c, GFS_OP_READ, fs.hfid, base, st, nb, 0, 0, nullptr, 0, nullptr);
     if (r < 0) {
       if (st >= 0) stage_free(c, st);
-      atom_or_rel(&c->f_state[g], GFS_ST_ERROR);
-      atom_and_rel(&c->f_state[g], ~GFS_ST_FILLING);
-      atom_add_rel(&c->f_state[g], 0xFFFFFFFFu);
+      a64_or_rel(&c->f_state[g], GFS_ST_ERROR);
+      a64_and_rel(&c->f_state[g], fl64(GFS_ST_FILLING));
+      a64_add_rel(&c->f_state[g], kRefDec);
       out.frame = r == -ETIMEDOUT ? r : -EIO;
       out.fill = 0;
       break;
@@ -941,16 +992,13 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
         sc.stage[tid] = -1;
         sc.fill[tid] = 0;
         st_rlx(&c->f_valid[f], sc.nbytes[tid]);
-        atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);  // publish the page
+        a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));  // publish the page
       }
     }
     if (err) {
       if (tid < (int)cnt && sc.frame[tid] >= 0) {
         const uint32_t f = (uint32_t)sc.frame[tid];
-        if (sc.fill[tid]) {  // an installed O_GWRONCE page nobody wrote: give it back
-          st_rel64(&c->f_tag[f], GFS_TAG_NONE);
-          atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
-        }
+        if (sc.fill[tid]) frame_retire(c, f, GFS_ST_FILLING);  // an installed O_GWRONCE page nobody wrote
         frame_release(c, f);
       }
       __syncthreads();
@@ -1011,17 +1059,17 @@ __device__ __forceinline__ bool snap_fd_cached(const gfs_ctx* c, Scratch& sc, in
 // Claim page p's frame for write-back if it is dirty and unreferenced.
 // Returns the frame (state EVICTING) or -1 (clean / absent), or -EBUSY.
 __device__ int claim_dirty(const gfs_ctx* c, const FileSnap& fs, uint64_t p) {
-  uint32_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
+  uint64_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
   if (!slot) return -1;
-  const uint32_t s = ld_acq(slot);
-  if (!s) return -1;
-  const uint32_t f = s - 1;
+  const uint64_t s = ld_acq64(slot);
+  if (!(uint32_t)s) return -1;
+  const uint32_t f = (uint32_t)s - 1u;
   const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
   if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) return -1;
-  if (atom_cas(&c->f_state[f], 0u, GFS_ST_EVICTING) != 0u)
+  if (!claim_frame(&c->f_state[f], 0u))
     return (ld_acq64(&c->f_tag[f]) == want && ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) ? -EBUSY : -1;
   if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) {
-    atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+    a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
     return -1;
   }
   return (int)f;
@@ -1041,7 +1089,7 @@ __device__ int sync_pages_lane(const gfs_ctx* c, const FileSnap& fs, uint64_t pb
     if (f < 0) continue;
     const int32_t r = frame_writeback_lane(c, (uint32_t)f, fs.hfid);
     if (r < 0) rc = r;
-    atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+    a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
   }
   return rc;
 }
@@ -1050,24 +1098,25 @@ __device__ int sync_pages_lane(const gfs_ctx* c, const FileSnap& fs, uint64_t pb
 __device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uint64_t pe, int tid, int nthr) {
   int rc = 0;
   for (uint64_t p = pb + tid; p < pe; p += nthr) {
-    uint32_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
+    uint64_t* slot = walk(c, fs.root, fs.height, p, false, nullptr);
     if (!slot) continue;
-    const uint32_t s = ld_acq(slot);
-    if (!s) continue;
-    const uint32_t f = s - 1;
+    const uint64_t s = ld_acq64(slot);
+    if (!(uint32_t)s) continue;
+    const uint32_t f = (uint32_t)s - 1u;
     const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
     if (ld_acq64(&c->f_tag[f]) != want) continue;
-    if (atom_cas(&c->f_state[f], 0u, GFS_ST_EVICTING) != 0u) {
+    if (!claim_frame(&c->f_state[f], 0u)) {
       rc = -EBUSY;
       continue;
     }
     if (ld_acq64(&c->f_tag[f]) == want) {
-      st_rlx64(&c->f_tag[f], GFS_TAG_NONE);
       st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
       st_rlx(&c->f_hi[f], 0);
       st_rlx(&c->f_written[f], 0);
+      frame_retire(c, f, GFS_ST_EVICTING);  // slots naming this generation go stale
+    } else {
+      a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
     }
-    atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
   }
   return rc;
 }
@@ -1171,11 +1220,12 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, int flags_in, Pre
       if (pst >= 0) {  // install page 0 while nobody else can see the file
         int ok = 0;
         const uint32_t nb = (uint32_t)rs.pad[0];
-        uint32_t* slot = nb ? walk(c, e->root, e->height, 0, true, nullptr) : nullptr;
+        uint64_t* slot = nb ? walk(c, e->root, e->height, 0, true, nullptr) : nullptr;
         if (slot) {
-          const int g = alloc_frame(c, (uint64_t)e->uid << 32, i);
+          uint32_t gen = 0;
+          const int g = alloc_frame(c, (uint64_t)e->uid << 32, i, &gen);
           if (g >= 0) {
-            if (atom_cas(slot, 0u, (uint32_t)g + 1u) == 0u) {
+            if (a64_cas(slot, 0ull, slot_val((uint32_t)g, gen)) == 0ull) {
               pf->frame = g;
               pf->stage = pst;
               pf->nbytes = nb;
@@ -1332,7 +1382,7 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
     if (tid == 0) {
       detail::stage_free(c, sc.stage[0]);
       detail::st_rlx(&c->f_valid[f], sc.nbytes[0]);
-      detail::atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+      detail::a64_and_rel(&c->f_state[f], detail::fl64(GFS_ST_FILLING));
       detail::frame_release(c, f);
       sc.frame[0] = -1;
     }
@@ -1393,6 +1443,7 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
     }
     __syncwarp(nthr >= 32 ? 0xFFFFFFFFu : ((1u << nthr) - 1u));
     const int64_t n0 = sc.ret;
+    uint32_t quick = 0;
     if (n0 > 0) {
       const uint64_t q0 = off >> shift, q1 = (off + (uint64_t)n0 - 1) >> shift;
       const uint32_t cnt = (uint32_t)((q1 - q0 + 1) < B ? (q1 - q0 + 1) : B);
@@ -1405,6 +1456,16 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
           sc.fill[tid] = r.fill;
           sc.stage[tid] = r.stage;
           sc.nbytes[tid] = r.nbytes;
+        } else if (q0 == q1 && n0 < (1 << 20) && __isShared(dst) && ((((uintptr_t)dst) | off | (uint64_t)n0) & 15) == 0 &&
+                   sc.mbar_grid == grid_id() && sc.mbar_blk == block_linear()) {
+          // Quick path: a one-page hit into shared memory. Lane 0 issues the
+          // TMA bulk copy now, before the block barrier, so the copy overlaps
+          // the other warps' arrival; they only wait on the mbarrier.
+          asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
+          mbar_expect_tx(&sc.mbar, (uint32_t)n0);
+          tma_load(dst, frame_ptr(c, (uint32_t)f) + (off & (P - 1)), (uint32_t)n0, &sc.mbar);
+          sc.frame[0] = f;
+          quick = 1;
         } else {
           sc.frame[tid] = f;
           sc.fill[tid] = 0;
@@ -1412,10 +1473,21 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
         }
       }
     }
+    if (tid == 0) sc.quick = quick;
   }
   __syncthreads();
   const int64_t n = sc.ret;
   if (n <= 0) return n;
+  if (sc.quick) {
+    const uint32_t ph = sc.mbar_phase;
+    mbar_wait(&sc.mbar, ph);
+    __syncthreads();
+    if (tid == 0) {
+      sc.mbar_phase = ph ^ 1u;
+      frame_release(c, (uint32_t)sc.frame[0]);
+    }
+    return n;
+  }
   const FileSnap fs = sc.fs;
   const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
   // TMA path: shared-memory destination, everything 16-byte aligned, the
@@ -1515,7 +1587,7 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
       atomicMin(&c->f_lo[f], s);
       atomicMax(&c->f_hi[f], e);
       atomicAdd(&c->f_written[f], e - s);
-      if (sc.fill[tid]) atom_and_rel(&c->f_state[f], ~GFS_ST_FILLING);
+      if (sc.fill[tid]) a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));
       frame_release_rel(c, f);
     }
   }
@@ -1564,7 +1636,7 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
           const int st = stage_alloc(c);
           sc.stage[tid] = st;
           if (st < 0) {
-            atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+            a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
             sc.frame[tid] = -1;
             atomicMin(&sc.err, st);
           }
@@ -1594,7 +1666,7 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
           ctr(c, GFS_C_RPC_WRITE);
           ctr(c, GFS_C_BYTES_D2H, hi - lo);
         }
-        atom_and_rel(&c->f_state[f], ~GFS_ST_EVICTING);
+        a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
       }
       __syncthreads();
     }

@@ -35,7 +35,11 @@ extern "C" {
 #define GFS_F_LOCKED_TRAVERSAL 1u /* K5 ablation: every lookup takes the file lock */
 #define GFS_F_NO_DMA_COMPLETION 2u /* fallback: completion via memcpy instead of stream write-value */
 
-/* ---- frame state word (pframe "state") ---------------------------------
+/* ---- frame state word (pframe "state", 64 bits) -------------------------
+ * bits 32..63 generation: +1 each time the frame is (re)assigned to a page.
+ *             Leaf slots of the radix tree hold (generation << 32) | (frame+1),
+ *             so one atomic increment both takes the reference and validates
+ *             the slot (no separate tag load; install CAS cannot ABA).
  * bits 0..23  reference count (gread/gwrite copies and gmmap mappings)
  * bit  24     FILLING  — frame installed, contents not yet valid
  * bit  25     EVICTING — claimed by eviction / gfsync / truncate (ref was 0)
@@ -152,7 +156,7 @@ typedef struct gfs_ctx {
   uint32_t nframes;
   uint8_t* pool;
   /* pframes, SoA */
-  uint32_t* f_state;
+  uint64_t* f_state;  /* generation << 32 | flags | refcount */
   uint64_t* f_tag;
   uint32_t* f_file;
   uint32_t* f_valid;
@@ -162,8 +166,8 @@ typedef struct gfs_ctx {
   uint32_t* f_stamp;
   uint32_t* fresh_next;
   uint32_t* hand;
-  /* radix node pool */
-  uint32_t* nodes;
+  /* radix node pool: 64-bit entries (interior: child node id; leaf: gen << 32 | frame + 1) */
+  uint64_t* nodes;
   uint32_t max_nodes;
   uint32_t max_files; /* power of two */
   uint32_t* node_next;

@@ -616,7 +616,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
     CK(cudaMalloc((void**)&c.pool, nframes * cfg->page_size));
     h->own_pool = true;
   }
-  CK(cudaMalloc((void**)&c.f_state, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_state, (size_t)nframes * 8));
   CK(cudaMalloc((void**)&c.f_tag, nframes * 8));
   CK(cudaMalloc((void**)&c.f_file, nframes * 4));
   CK(cudaMalloc((void**)&c.f_valid, nframes * 4));
@@ -627,7 +627,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMalloc((void**)&c.fresh_next, 4));
   CK(cudaMalloc((void**)&c.hand, 4));
   c.max_nodes = max_nodes;
-  CK(cudaMalloc((void**)&c.nodes, (size_t)max_nodes * GFS_FANOUT * 4));
+  CK(cudaMalloc((void**)&c.nodes, (size_t)max_nodes * GFS_FANOUT * 8));
   CK(cudaMalloc((void**)&c.node_next, 4));
   CK(cudaMalloc((void**)&c.node_free, (size_t)max_nodes * 4));
   CK(cudaMalloc((void**)&c.node_free_top, 4));
@@ -660,7 +660,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   c.flags = cfg->flags;
   c.max_batch = cfg->max_batch >= 1 && cfg->max_batch <= GFS_MAX_BATCH ? cfg->max_batch : GFS_MAX_BATCH;
   c.timeout_ns = cfg->timeout_ms * 1000000ull;
-  CK(cudaMemsetAsync(c.nodes, 0, (size_t)max_nodes * GFS_FANOUT * 4, h->priv));
+  CK(cudaMemsetAsync(c.nodes, 0, (size_t)max_nodes * GFS_FANOUT * 8, h->priv));
   CK(cudaMemsetAsync(c.files, 0, (size_t)MF * sizeof(gfs_file), h->priv));
   CK(cudaMemsetAsync(c.paths, 0, (size_t)MF * GFS_MAX_PATH, h->priv));
   CK(cudaMemsetAsync(c.staging_bits, 0, (size_t)words * 4, h->priv));

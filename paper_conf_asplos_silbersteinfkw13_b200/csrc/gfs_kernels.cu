@@ -25,7 +25,7 @@ namespace {
 __global__ void k_init_metadata(gfs_ctx c) {
   const size_t stride = (size_t)gridDim.x * blockDim.x;
   for (size_t i = blockIdx.x * (size_t)blockDim.x + threadIdx.x; i < c.nframes; i += stride) {
-    c.f_state[i] = GFS_ST_EVICTING;  // never-used frames are handed out by fresh_next only
+    c.f_state[i] = (uint64_t)GFS_ST_EVICTING;  // never-used frames are handed out by fresh_next only
     c.f_tag[i] = GFS_TAG_NONE;
     c.f_file[i] = 0xFFFFFFFFu;
     c.f_valid[i] = 0;
