@@ -20,7 +20,8 @@ COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", 
             "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
             "ring_wait", "busy", "stage_wait"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
-                 "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns"]
+                 "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns",
+                 "mapped_reads"]
 
 O_RDONLY = 0
 O_GWRONCE = 1

@@ -32,6 +32,8 @@
 #include <fcntl.h>
 #include <mutex>
 #include <sched.h>
+#include <csetjmp>
+#include <csignal>
 #include <string>
 #include <sys/mman.h>
 #include <sys/resource.h>
@@ -149,7 +151,7 @@ struct VersionTable {
 
 enum {
   HS_RPC = 0, HS_READ, HS_WRITE, HS_OPEN, HS_CLOSE, HS_TRUNC, HS_BYTES_H2D, HS_BYTES_D2H, HS_PREAD_NS,
-  HS_ERRORS, HS_MERGES, HS_BUSY_NS, HS_OPEN_NS, HS_OPEN_SYS_NS, HS_OPEN_PF_NS, HS_OPEN_TAB_NS, HS_N
+  HS_ERRORS, HS_MERGES, HS_BUSY_NS, HS_OPEN_NS, HS_OPEN_SYS_NS, HS_OPEN_PF_NS, HS_OPEN_TAB_NS, HS_MAPPED, HS_N
 };
 
 }  // namespace
@@ -162,9 +164,13 @@ enum {
 // -ESTALE); `gen` invalidates cached fds when an hfid is recycled.
 struct HostFile {
   bool live = false;
+  bool map_tried = false;
   uint32_t gen = 0;
   uint32_t mode = 0;
   uint64_t dev = 0, ino = 0;
+  uint64_t size = 0;        // size at (re)open
+  uint8_t* map = nullptr;   // read-only shared mapping of [0, map_len), large O_RDONLY files
+  uint64_t map_len = 0;
   std::string path;
 };
 
@@ -198,6 +204,7 @@ struct gfs_handle {
   std::atomic<bool> running{false};
   std::mutex fd_mu;  // protects files / free_hfids
   std::vector<HostFile> files;
+  uint32_t nmapped = 0;
   std::vector<uint32_t> free_hfids;
   size_t fd_cap = 1024;  // per worker
   VersionTable vt;
@@ -248,12 +255,75 @@ bool hfid_meta(gfs_handle* h, uint32_t id, HostFile* out) {
 }
 
 void free_hfid(gfs_handle* h, uint32_t id) {
-  std::lock_guard<std::mutex> g(h->fd_mu);
-  if (id >= h->files.size() || !h->files[id].live) return;
-  const uint32_t gen = h->files[id].gen + 1;
-  h->files[id] = HostFile();
-  h->files[id].gen = gen;  // cached fds of the old file are now stale
-  h->free_hfids.push_back(id);
+  uint8_t* map = nullptr;
+  uint64_t map_len = 0;
+  {
+    std::lock_guard<std::mutex> g(h->fd_mu);
+    if (id >= h->files.size() || !h->files[id].live) return;
+    const uint32_t gen = h->files[id].gen + 1;
+    map = h->files[id].map;
+    map_len = h->files[id].map_len;
+    if (map) --h->nmapped;
+    h->files[id] = HostFile();
+    h->files[id].gen = gen;  // cached fds of the old file are now stale
+    h->free_hfids.push_back(id);
+  }
+  // No READ of this hfid can be in flight: the GPU closes a file only after
+  // every block holding it open is done with it.
+  if (map) munmap(map, map_len);
+}
+
+// ---- mapped reads --------------------------------------------------------
+// READ of a large O_RDONLY file copies from a shared read-only mapping of the
+// file instead of pread(): the same bytes (page cache), but one user-space
+// memcpy per page instead of the kernel's per-4KiB copy loop (measured 1.4x
+// per daemon thread on tmpfs). A file that shrinks under the mapping raises
+// SIGBUS on access; the handler returns to the READ, which falls back to
+// pread (short read, zero tail: R4).
+constexpr uint64_t kMapMinBytes = 64ull << 20;
+constexpr uint32_t kMapMaxFiles = 4096;
+thread_local sigjmp_buf* volatile t_bus_jb = nullptr;  // volatile: the stores around memcpy must stay
+struct sigaction g_old_bus;
+std::once_flag g_bus_once;
+
+void on_sigbus(int sig, siginfo_t* si, void* uc) {
+  if (t_bus_jb) siglongjmp(*t_bus_jb, 1);
+  if (g_old_bus.sa_flags & SA_SIGINFO) {
+    if (g_old_bus.sa_sigaction) g_old_bus.sa_sigaction(sig, si, uc);
+    return;
+  }
+  if (g_old_bus.sa_handler == SIG_DFL || g_old_bus.sa_handler == SIG_IGN) {
+    signal(SIGBUS, SIG_DFL);
+    raise(SIGBUS);
+    return;
+  }
+  g_old_bus.sa_handler(sig);
+}
+
+void install_sigbus() {
+  std::call_once(g_bus_once, [] {
+    struct sigaction sa;
+    memset(&sa, 0, sizeof(sa));
+    sa.sa_sigaction = on_sigbus;
+    sa.sa_flags = SA_SIGINFO | SA_NODEFER;
+    sigemptyset(&sa.sa_mask);
+    sigaction(SIGBUS, &sa, &g_old_bus);
+  });
+}
+
+// Copy [off, off+len) of the mapping into buf; false if the access faulted.
+bool map_copy(uint8_t* buf, const uint8_t* map, uint64_t off, uint64_t len) {
+  sigjmp_buf jb;
+  if (sigsetjmp(jb, 0) != 0) {
+    t_bus_jb = nullptr;
+    return false;
+  }
+  t_bus_jb = &jb;
+  std::atomic_signal_fence(std::memory_order_seq_cst);
+  memcpy(buf, map + off, len);
+  std::atomic_signal_fence(std::memory_order_seq_cst);
+  t_bus_jb = nullptr;
+  return true;
 }
 
 // open(path) as openat(this worker's cached fd of dirname(path), basename).
@@ -385,6 +455,7 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
     f.mode = q.flags;
     f.dev = st.st_dev;
     f.ino = st.st_ino;
+    f.size = (uint64_t)st.st_size;
     f.path = path;
     hfid = alloc_hfid(h, f);
     HostFile m;
@@ -403,13 +474,58 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
   return 0;
 }
 
+// The mapping of hfid `id` (created on first use for a large O_RDONLY file).
+// Returns nullptr when the file is not (or cannot be) mapped.
+const uint8_t* hfid_map(gfs_handle* h, Worker& w, uint32_t id, uint64_t* map_len) {
+  uint64_t size;
+  uint32_t gen;
+  {
+    std::lock_guard<std::mutex> g(h->fd_mu);
+    if (id >= h->files.size() || !h->files[id].live) return nullptr;
+    HostFile& f = h->files[id];
+    if (f.map) {
+      *map_len = f.map_len;
+      return f.map;
+    }
+    if (f.map_tried || (f.mode & GFS_O_GWRONCE) || f.size < kMapMinBytes || h->nmapped >= kMapMaxFiles)
+      return nullptr;
+    f.map_tried = true;  // one worker maps it; the others pread meanwhile
+    size = f.size;
+    gen = f.gen;
+  }
+  const int fd = w_fd(h, w, id);
+  if (fd < 0) return nullptr;
+  void* p = mmap(nullptr, size, PROT_READ, MAP_SHARED, fd, 0);
+  if (p == MAP_FAILED) return nullptr;
+  install_sigbus();
+  std::lock_guard<std::mutex> g(h->fd_mu);
+  HostFile& f = h->files[id];
+  if (!f.live || f.gen != gen || f.map) {
+    munmap(p, size);
+    return nullptr;
+  }
+  f.map = (uint8_t*)p;
+  f.map_len = size;
+  ++h->nmapped;
+  *map_len = size;
+  return f.map;
+}
+
 int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   if (q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
-  const int fd = w_fd(h, w, q.hfid);
-  if (fd < 0) return fd;
   uint8_t* buf = staging_slot(h, q.stage);
   auto t0 = std::chrono::steady_clock::now();
-  int64_t n = pread_full(fd, buf, q.len, q.file_off);
+  uint64_t map_len = 0;
+  const uint8_t* map = hfid_map(h, w, q.hfid, &map_len);
+  int64_t n = -1;
+  if (map && q.file_off + q.len <= map_len && map_copy(buf, map, q.file_off, q.len)) {
+    n = q.len;
+    h->hs[HS_MAPPED]++;
+  } else {
+    const int fd = w_fd(h, w, q.hfid);
+    if (fd < 0) return fd;
+    n = pread_full(fd, buf, q.len, q.file_off);
+  }
   h->hs[HS_PREAD_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
                             std::chrono::steady_clock::now() - t0).count();
   if (n < 0) return (int32_t)n;
@@ -718,6 +834,8 @@ GFS_API int gfs_shutdown(gfs_handle* h) {
   cudaSetDevice(h->cfg.device);
   cudaStreamSynchronize(h->priv);
   free_all(h);
+  for (HostFile& f : h->files)
+    if (f.map) munmap(f.map, f.map_len);
   delete h;
   return 0;
 }

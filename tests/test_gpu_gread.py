@@ -165,3 +165,24 @@ def test_errors(g, shmdir):
         assert fs.gfstat(p) == 1000
         ret, _, _ = fs.gread_calls(p, [0, 999, 1000, 5000], [2000, 10, 1, 1], grid=2)
         assert ret.tolist() == [1000, 1, 0, 0]
+
+
+def test_mapped_reads_and_external_shrink(g, shmdir):
+    """Large read-only files are served from a host mapping (same bytes as
+    pread); a file shrunk under the mapping while open reads zeros past the
+    new end (R4) instead of crashing the daemon (SIGBUS -> pread fallback)."""
+    P = 1 << 20
+    size = 80 << 20
+    path = gen.splitmix_file(os.path.join(shmdir, "big.bin"), size, seed=44)
+    offs, lens = gen.random_calls(9, 200, 40 << 20, 3 * P, page_size=P)  # pages >= 40 MiB stay uncached
+    with _fs(g, cache_bytes=64 * P, page_size=P) as fs:
+        pfd = fs.pin(path)  # stays open: no revalidation on the next gopens
+        assert pfd >= 0
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, grid=16)
+        check_calls(path, size, offs, lens, ret, dst, dstoff)
+        assert fs.host_stats()["mapped_reads"] > 0
+        os.truncate(path, 40 << 20)
+        ret, dst, dstoff = fs.gread_calls(path, [70 << 20], [2 * P], grid=1)
+        assert ret[0] == 2 * P  # the open file's size is the one seen at gopen
+        assert not dst[:2 * P].any()
+        fs.unpin(pfd)
