@@ -378,7 +378,7 @@ def grep_phase(args, torch, g, gen, dev, stream, hbm, rank, ws, local, dist):
             with torch.cuda.stream(stream):
                 e0.record(stream)
                 st = fs.grep(c["dict"], lst, hits=False, keep_open=True, stream=stream, sync=False, state=state,
-                             pair_cap=1 << 24)
+                             rec_cap=1 << 24)
                 e1.record(stream)
                 stream.synchronize()
             state = st

@@ -99,6 +99,8 @@ int gfs_info(gfs_handle* h, uint64_t* out, int n);
  *           d_dst + d_dstoff[i]; gmunmap; d_ret[i] = p ? m : -errno-or-0
  *   mode 2: like mode 0 but the destination is dynamic shared memory
  *           (requires d_len[i] <= smem_bytes), copied out to d_dst afterwards
+ *   mode 3: like mode 2 with the destination at smem + d_off[i] % 16, i.e.
+ *           co-aligned with the file offset (requires d_len[i] + 15 <= smem_bytes)
  * then gclose(). If gopen fails every d_ret[i] of that block gets its error. */
 int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
                   const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,

@@ -602,6 +602,46 @@ __device__ __forceinline__ void mbar_wait(uint64_t* m, uint32_t phase) {
       : "memory");
 }
 
+// The block's mbarrier lives in `Scratch` (static shared memory, not cleared
+// between launches): (re)initialise it the first time this block of this launch
+// needs it. Called by thread 0 only, before the barrier that publishes it.
+__device__ __forceinline__ void ensure_mbar(Scratch& sc) {
+  if (sc.mbar_grid != grid_id() || sc.mbar_blk != block_linear()) {
+    mbar_init(&sc.mbar);
+    sc.mbar_phase = 0;
+    sc.mbar_grid = grid_id();
+    sc.mbar_blk = block_linear();
+  }
+}
+
+// TMA bulk copy of one co-aligned span ((dst - src) % 16 == 0): the 16-byte
+// aligned middle goes through cp.async.bulk, the <16-byte head and tail are
+// left to copy_edges(). Returns the bytes the mbarrier must expect.
+__device__ __forceinline__ uint32_t span_mid(const uint8_t* src, uint32_t n) {
+  const uint32_t h0 = (16u - ((uint32_t)(uintptr_t)src & 15u)) & 15u;
+  return (n - (h0 < n ? h0 : n)) & ~15u;
+}
+__device__ __forceinline__ uint32_t tma_span(uint8_t* dst, const uint8_t* src, uint32_t n, uint64_t* m) {
+  const uint32_t h0 = (16u - ((uint32_t)(uintptr_t)src & 15u)) & 15u;
+  const uint32_t head = h0 < n ? h0 : n;
+  const uint32_t mid = (n - head) & ~15u;
+  if (mid) tma_load(dst + head, src + head, mid, m);
+  return mid;
+}
+
+// The head and tail bytes tma_span() leaves out, copied by threads tid < 32.
+__device__ __forceinline__ void copy_edges(uint8_t* dst, const uint8_t* src, uint32_t n, int tid) {
+  const uint32_t h0 = (16u - ((uint32_t)(uintptr_t)src & 15u)) & 15u;
+  const uint32_t head = h0 < n ? h0 : n;
+  const uint32_t mid = (n - head) & ~15u;
+  const uint32_t tail = n - head - mid;
+  if (tid < (int)head) dst[tid] = __ldcg(src + tid);
+  else if (tid < (int)(head + tail)) {
+    const uint32_t k = head + mid + (uint32_t)tid - head;
+    dst[k] = __ldcg(src + k);
+  }
+}
+
 // ------------------------------------------------------------------ frames
 __device__ __forceinline__ uint8_t* frame_ptr(const gfs_ctx* c, uint32_t f) {
   return c->pool + ((size_t)f << c->page_shift);
@@ -1365,12 +1405,7 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
       sc.cached_fd = fd;
       for (int i = 0; i < detail::kLeafCache; ++i) sc.leaf[i] = 0;
     }
-    if (sc.mbar_grid != detail::grid_id() || sc.mbar_blk != detail::block_linear()) {
-      detail::mbar_init(&sc.mbar);  // first gopen of this block in this launch
-      sc.mbar_phase = 0;
-      sc.mbar_grid = detail::grid_id();
-      sc.mbar_blk = detail::block_linear();
-    }
+    detail::ensure_mbar(sc);
   }
   __syncthreads();
   if (sc.frame[0] >= 0) {  // pull the prefetched page 0 and publish it
@@ -1428,6 +1463,7 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   // (one page per lane). Other warps only touch `sc` after the next barrier.
   if (tid < 32) {
     if (tid == 0) {
+      ensure_mbar(sc);
       FileSnap s;
       const bool cached = sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id();
       if (cached) s = sc.cached;
@@ -1456,14 +1492,16 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
           sc.fill[tid] = r.fill;
           sc.stage[tid] = r.stage;
           sc.nbytes[tid] = r.nbytes;
-        } else if (q0 == q1 && n0 < (1 << 20) && __isShared(dst) && ((((uintptr_t)dst) | off | (uint64_t)n0) & 15) == 0 &&
-                   sc.mbar_grid == grid_id() && sc.mbar_blk == block_linear()) {
+        } else if (q0 == q1 && n0 < (1 << 20) && __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0) {
           // Quick path: a one-page hit into shared memory. Lane 0 issues the
-          // TMA bulk copy now, before the block barrier, so the copy overlaps
-          // the other warps' arrival; they only wait on the mbarrier.
+          // TMA bulk copy of the aligned middle now, before the block barrier,
+          // so the copy overlaps the other warps' arrival; they only wait on
+          // the mbarrier (head/tail bytes are copied by warp 0 after it).
           asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
-          mbar_expect_tx(&sc.mbar, (uint32_t)n0);
-          tma_load(dst, frame_ptr(c, (uint32_t)f) + (off & (P - 1)), (uint32_t)n0, &sc.mbar);
+          uint64_t* mb = &sc.mbar;
+          const uint8_t* src = frame_ptr(c, (uint32_t)f) + (off & (P - 1));
+          mbar_expect_tx(mb, span_mid(src, (uint32_t)n0));
+          tma_span((uint8_t*)dst, src, (uint32_t)n0, mb);
           sc.frame[0] = f;
           quick = 1;
         } else {
@@ -1480,6 +1518,7 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   if (n <= 0) return n;
   if (sc.quick) {
     const uint32_t ph = sc.mbar_phase;
+    copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + (off & (P - 1)), (uint32_t)n, tid);
     mbar_wait(&sc.mbar, ph);
     __syncthreads();
     if (tid == 0) {
@@ -1490,10 +1529,10 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   }
   const FileSnap fs = sc.fs;
   const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
-  // TMA path: shared-memory destination, everything 16-byte aligned, the
-  // block's mbarrier initialised in this launch (set up by its gopen).
-  const bool tma = __isShared(dst) && ((((uintptr_t)dst) | off | (uint64_t)n) & 15) == 0 &&
-                   sc.mbar_grid == grid_id() && sc.mbar_blk == block_linear();
+  // TMA path: shared-memory destination co-aligned with the file offset
+  // ((dst - off) % 16 == 0, so frame and destination agree mod 16): aligned
+  // middles by TMA, the call's head and tail bytes by warp 0.
+  const bool tma = __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0;
   for (uint64_t pb = p0; pb <= p1; pb += B) {
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
     const int err = acquire_batch(c, sc, fs, pb, cnt, pb == p0);
@@ -1505,13 +1544,30 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
       const uint32_t ph = sc.mbar_phase;
       if (tid == 0) {
         asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
-        mbar_expect_tx(&sc.mbar, (uint32_t)batch_bytes);
+        uint32_t tx = 0;
+        for (uint32_t i = 0; i < cnt; ++i) {  // interior pages are whole and aligned: only the
+          const uint64_t p = pb + i;          // call's first and last pages have edges
+          const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+          const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+          tx += span_mid(frame_ptr(c, (uint32_t)sc.frame[i]) + s, (uint32_t)(e - s));
+        }
+        mbar_expect_tx(&sc.mbar, tx);
         for (uint32_t i = 0; i < cnt; ++i) {
           const uint64_t p = pb + i;
           const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
           const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-          tma_load((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+          tma_span((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
                    (uint32_t)(e - s), &sc.mbar);
+        }
+      }
+      if (tid < 32) {
+        if (pb == p0) {
+          const uint64_t s = off & (P - 1), e = p0 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+          copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + s, (uint32_t)(e - s), tid);
+        }
+        if (pb + cnt - 1 == p1 && p1 != p0) {
+          const uint64_t e = ((off + (uint64_t)n - 1) & (P - 1)) + 1;
+          copy_edges((uint8_t*)dst + ((p1 << shift) - off), frame_ptr(c, (uint32_t)sc.frame[cnt - 1]), (uint32_t)e, tid);
         }
       }
       mbar_wait(&sc.mbar, ph);

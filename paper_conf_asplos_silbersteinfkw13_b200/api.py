@@ -80,7 +80,8 @@ class GpuFS:
 
     # gread / gmmap parity harness -------------------------------------------
     def gread_calls(self, path, offs, lens, mode=0, grid=None, block=256, smem=0, stream=None):
-        """Issue gread (mode 0), gmmap (1) or gread-to-shared (2) calls; returns (ret, dst, dstoff)."""
+        """Issue gread (mode 0), gmmap (1), gread-to-shared (2) or gread-to-shared co-aligned with the
+        offset (3) calls; returns (ret, dst, dstoff)."""
         torch = _torch()
         offs = np.asarray(offs, dtype=np.uint64)
         lens = np.asarray(lens, dtype=np.uint64)
@@ -94,7 +95,7 @@ class GpuFS:
         d_ret = torch.full((max(n, 1),), -999, dtype=torch.int64, device=f"cuda:{self.device}")
         s, sp = self._stream(stream)
         grid = grid or max(1, min(n, 296))
-        if mode == 2 and smem == 0:
+        if mode >= 2 and smem == 0:
             smem = int(lens.max()) if n else 16
             smem = (smem + 15) // 16 * 16
         gfs_run_gread(self.h, sp, path, mode, n, d_off.data_ptr(), d_len.data_ptr(), d_dstoff.data_ptr(),
@@ -173,8 +174,9 @@ class GpuFS:
         return int(d_ret.item())
 
     # grep -w ------------------------------------------------------------------
-    def grep(self, dict_path, list_path, hits=False, chunk=16384, grid=None, block=256, keep_open=False,
-             pair_cap=1 << 22, hit_cap=None, stream=None, sync=True, state=None, corpus_cap=1 << 34):
+    def grep(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
+             pair_cap=1 << 24, hit_cap=None, stream=None, sync=True, state=None, corpus_cap=1 << 34,
+             rec_cap=1 << 22):
         """grep -w. Returns a dict with records (n,3) sorted by (file, word),
         totals, digest (sum, xor, nhits), hits (n,3) sorted by (file, offset, word) if requested.
 
@@ -188,20 +190,20 @@ class GpuFS:
             nwords = max(1, os.path.getsize(dict_path) // 32)
             lbytes = os.path.getsize(list_path)
             p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
-                                pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 4 * 148, block=block,
+                                pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 1 << 20, block=block,
                                 keep_open=1 if keep_open else 0, corpus_cap=corpus_cap)
             if hits:
                 p.hit_cap = hit_cap if hit_cap is not None else 1 << 22
             work = torch.empty(gfs_grep_work_bytes(p), dtype=torch.uint8, device=dev)
-            rec = torch.empty(3 * p.pair_cap, dtype=torch.int32, device=dev)
+            rec = torch.empty(3 * rec_cap, dtype=torch.int32, device=dev)
             totals = torch.empty(nwords, dtype=torch.int64, device=dev)
             d_hits = torch.empty(2 * max(p.hit_cap, 1), dtype=torch.int64, device=dev) if hits else None
             summ = torch.zeros(10, dtype=torch.int64, device=dev)
-            state = dict(p=p, work=work, rec=rec, totals=totals, hits=d_hits, summary=summ)
+            state = dict(p=p, work=work, rec=rec, rec_cap=rec_cap, totals=totals, hits=d_hits, summary=summ)
         p = state["p"]
         s, sp = self._stream(stream)
         gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
-                 p.pair_cap, state["totals"].data_ptr(),
+                 state["rec_cap"], state["totals"].data_ptr(),
                  state["hits"].data_ptr() if state["hits"] is not None else None, state["summary"].data_ptr())
         if not sync:
             return state
@@ -209,9 +211,9 @@ class GpuFS:
         summ = dict(zip(GREP_SUMMARY, (int(x) for x in state["summary"].cpu().numpy())))
         if summ["err"] == -28 and pair_cap < (1 << 30):  # -ENOSPC: a table was too small
             return self.grep(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap * 4, hit_cap,
-                             stream, sync, None, corpus_cap * 4)
+                             stream, sync, None, corpus_cap * 4, max(rec_cap, summ["nrecords"]) * 2)
         out = {"summary": summ}
-        nrec = min(summ["nrecords"], p.pair_cap)
+        nrec = min(summ["nrecords"], state["rec_cap"])
         r = state["rec"][:3 * nrec].view(nrec, 3).cpu().numpy().astype(np.uint64)
         order = np.lexsort((r[:, 1], r[:, 0])) if nrec else np.zeros(0, np.int64)
         out["records"] = r[order]

@@ -16,12 +16,17 @@
 //   k_grep_open   gopen every file once (first gopen goes to the host,
 //                 P:L370-372), record fd and size;
 //   k_grep_plan   exclusive scan of per-file work-item counts, item -> file map;
-//   k_grep_scan   persistent blocks pull items (file, chunk): gread the chunk
-//                 plus a halo into shared memory; pass 1 compacts token starts
-//                 (W(t[i]) and not W(t[i-1])) into a shared list, pass 2 gives
-//                 every thread whole tokens (no divergence between lanes): hash +
-//                 probe tokens of <= 32 bytes, count matches per item in shared
-//                 memory, flush (file, word) counts into a global table;
+//   k_grep_scan   persistent blocks pull items: a whole file when it fits one
+//                 item, else a chunk of it. gread brings the item plus a halo
+//                 into shared memory (TMA). Pass 1 classifies 32-byte stripes
+//                 into word-byte bit masks (SWAR, 4 bytes per op); pass 2 gives
+//                 each thread the tokens that start in its stripe: length from
+//                 the masks, bytes gathered as 8 zero-padded words, one 64-bit
+//                 hash, one probe of the (L2-resident) table, an exact 32-byte
+//                 compare on a fingerprint match. Counts per item in shared
+//                 memory; a whole-file item emits its (file, word, count)
+//                 records directly, chunks of large files merge through a
+//                 global (file, word) table;
 //   k_grep_close  gclose every file (unless kept open for warm re-runs);
 //   k_grep_compact emit unique (file, word, count) records and word totals.
 // Word bytes are [A-Za-z0-9_] (GNU grep -w under LC_ALL=C, R10).
@@ -45,8 +50,10 @@ namespace {
 constexpr uint32_t kMaxPath = GFS_MAX_PATH;
 constexpr uint32_t kHalo = 48;      // bytes after the chunk: a token starting inside may run 33 bytes
 constexpr uint32_t kPre = 16;       // bytes before the chunk (one needed for the boundary test)
+constexpr uint32_t kSlack = 64;     // gathers read up to 48 bytes past a token start
 constexpr uint32_t kCountSlots = 2048;
-constexpr uint32_t kListChunk = 65536;
+constexpr uint32_t kListRead = 65536;  // list file gread granularity
+constexpr uint32_t kListChunk = 4096;  // list parse granularity (one block per chunk)
 constexpr uint64_t kPairEmpty = ~0ull;
 constexpr uint64_t kDupBit = 1ull << 63;  // table entry: the word has duplicates
 
@@ -67,8 +74,8 @@ struct GrepWork {
   uint32_t* item_file;    // item -> file
   uint64_t max_items;
   // (file, word) -> count table
-  uint64_t* pair_key;
-  uint64_t* pair_cnt;
+  uint64_t* pair;         // slot i: pair[2i] = (file << 32) | word (or empty), pair[2i+1] = count;
+                          // key and count share one 32-byte sector
   uint64_t pair_mask;
   // counters
   unsigned long long* vars;  // see V_*
@@ -80,12 +87,58 @@ __device__ __forceinline__ bool is_word(uint32_t ch) {
   return (ch - 'a' < 26u) || (ch - 'A' < 26u) || (ch - '0' < 10u) || ch == '_';
 }
 
-__device__ __forceinline__ uint64_t tok_hash(const uint8_t* p, uint32_t n) {
-  uint64_t h = 0xcbf29ce484222325ull;
-  for (uint32_t i = 0; i < n; ++i) h = (h ^ p[i]) * 0x100000001b3ull;
-  h ^= h >> 29;
-  h *= 0xbf58476d1ce4e5b9ull;
+// Word-byte mask of 4 bytes (SWAR): bit 7 of each byte set iff it is in
+// [A-Za-z0-9_]. in_range(x, lo, hi) per byte for x, lo, hi <= 0x7f:
+// (0x80 + x - lo) has bit 7 iff x >= lo, (0x80 + hi - x) iff x <= hi, and
+// neither subtraction borrows across bytes. Bytes >= 0x80 are non-word.
+__device__ __forceinline__ uint32_t word_bits4(uint32_t x) {
+  constexpr uint32_t H = 0x80808080u, O = 0x01010101u;
+  const uint32_t x7 = x & 0x7F7F7F7Fu;
+  const uint32_t l = x7 | 0x20202020u;  // fold A-Z onto a-z
+  const uint32_t alpha = ((l | H) - 0x61u * O) & ((0x7Au | 0x80u) * O - l);
+  const uint32_t digit = ((x7 | H) - 0x30u * O) & ((0x39u | 0x80u) * O - x7);
+  const uint32_t under = ((x7 | H) - 0x5Fu * O) & ((0x5Fu | 0x80u) * O - x7);
+  const uint32_t m = (alpha | digit | under) & ~x & H;
+  // bits 7,15,23,31 -> 0..3 (the four partial products never overlap)
+  return (((m >> 7) * 0x00204081u) >> 21) & 0xFu;
+}
+
+// 32-bit word-byte mask of 32 bytes at p (16-byte aligned shared memory).
+__device__ __forceinline__ uint32_t word_bits32(const uint8_t* p) {
+  const uint4 a = *(const uint4*)p, b = *(const uint4*)(p + 16);
+  return word_bits4(a.x) | (word_bits4(a.y) << 4) | (word_bits4(a.z) << 8) | (word_bits4(a.w) << 12) |
+         (word_bits4(b.x) << 16) | (word_bits4(b.y) << 20) | (word_bits4(b.z) << 24) | (word_bits4(b.w) << 28);
+}
+
+// Hash of a word given as 8 little-endian 32-bit words, zero-padded past its
+// length L (dictionary slots and tokens are both brought to this form).
+__device__ __forceinline__ uint64_t tok_hash(const uint32_t (&v)[8], uint32_t L) {
+  uint64_t h = 0x9E3779B97F4A7C15ull * (L + 1);
+#pragma unroll
+  for (int j = 0; j < 4; ++j) {
+    h ^= ((uint64_t)v[2 * j + 1] << 32) | v[2 * j];
+    h *= 0xBF58476D1CE4E5B9ull;
+    h ^= h >> 29;
+  }
+  h *= 0x94D049BB133111EBull;
   return h ^ (h >> 32);
+}
+
+// Bytes [0, L) of the 32 starting at byte offset `sh` (0..15) of 12 words,
+// as 8 zero-padded words: two select levels + a funnel shift, no local memory.
+__device__ __forceinline__ void gather_token(const uint32_t (&W)[12], uint32_t sh, uint32_t L, uint32_t (&v)[8]) {
+  uint32_t A[10], B[9];
+#pragma unroll
+  for (int j = 0; j < 10; ++j) A[j] = (sh & 8) ? W[j + 2] : W[j];
+#pragma unroll
+  for (int j = 0; j < 9; ++j) B[j] = (sh & 4) ? A[j + 1] : A[j];
+  const uint32_t r = (sh & 3) * 8;
+#pragma unroll
+  for (int j = 0; j < 8; ++j) {
+    const uint32_t wv = __funnelshift_r(B[j], B[j + 1], r);
+    const int nb = min(max((int)L - 4 * j, 0), 4);
+    v[j] = wv & __funnelshift_lc(0xFFFFFFFFu, 0u, 8 * nb);  // low nb bytes
+  }
 }
 
 // entry bits 32..62 hold a 31-bit fingerprint, 26..31 the length
@@ -134,7 +187,7 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
       if (tid == 0) set_err(w, r < 0 ? r : -EIO);
     } else {
       for (uint32_t k = k0 + tid; k < k1; k += blockDim.x) {
-        const uint8_t* s = w.dict + (size_t)k * 32;
+        uint8_t* s = w.dict + (size_t)k * 32;
         uint32_t n = 0;
         while (n < 32 && s[n]) ++n;
         bool ok = n > 0;
@@ -143,7 +196,13 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
           set_err(w, -EINVAL);
           continue;
         }
-        const uint64_t h = tok_hash(s, n);
+        // zero the bytes after the word: the slot becomes the word's padded form
+        // (other threads only ever read bytes [0, n) of a slot of length n)
+        for (uint32_t i = n; i < 32; ++i) s[i] = 0;
+        uint32_t v[8];
+#pragma unroll
+        for (int j = 0; j < 8; ++j) v[j] = ((const uint32_t*)s)[j];
+        const uint64_t h = tok_hash(v, n);
         const uint64_t ent = entry_key(h, n) | (k + 1);
         uint32_t slot = (uint32_t)h & w.table_mask;
         for (uint32_t probe = 0; probe <= w.table_mask; ++probe, slot = (slot + 1) & w.table_mask) {
@@ -168,7 +227,7 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
 }
 
 // --------------------------------------------------------------- file list
-// Pass 1: every block greads its 64 KiB chunks of the list file.
+// Pass 1: every block greads its 64 KiB pieces of the list file.
 __global__ void k_grep_list_read(const gfs_ctx* c, const char* list_path, GrepWork w, uint64_t list_cap) {
   const int fd = gopen(c, list_path, GFS_O_RDONLY);
   if (fd < 0) {
@@ -180,8 +239,8 @@ __global__ void k_grep_list_read(const gfs_ctx* c, const char* list_path, GrepWo
     if (threadIdx.x == 0 && blockIdx.x == 0) set_err(w, -ENOSPC);
   } else {
     if (threadIdx.x == 0 && blockIdx.x == 0) w.vars[V_LISTSZ] = (unsigned long long)size;
-    for (uint64_t o = (uint64_t)blockIdx.x * kListChunk; o < (uint64_t)size; o += (uint64_t)gridDim.x * kListChunk) {
-      const uint64_t n = min((uint64_t)kListChunk, (uint64_t)size - o);
+    for (uint64_t o = (uint64_t)blockIdx.x * kListRead; o < (uint64_t)size; o += (uint64_t)gridDim.x * kListRead) {
+      const uint64_t n = min((uint64_t)kListRead, (uint64_t)size - o);
       const int64_t r = gread(c, fd, o, n, w.list + o);
       if (r != (int64_t)n && threadIdx.x == 0) set_err(w, r < 0 ? r : -EIO);
     }
@@ -352,10 +411,10 @@ __device__ __forceinline__ void pair_add(GrepWork& w, uint32_t f, uint32_t k, ui
   const uint64_t key = ((uint64_t)f << 32) | k;
   uint64_t slot = splitmix64(key) & w.pair_mask;
   for (uint64_t probe = 0; probe <= w.pair_mask; ++probe, slot = (slot + 1) & w.pair_mask) {
-    unsigned long long cur = atomicCAS((unsigned long long*)&w.pair_key[slot], (unsigned long long)kPairEmpty,
+    unsigned long long cur = atomicCAS((unsigned long long*)&w.pair[2 * slot], (unsigned long long)kPairEmpty,
                                        (unsigned long long)key);
     if (cur == kPairEmpty || cur == key) {
-      atomicAdd((unsigned long long*)&w.pair_cnt[slot], (unsigned long long)cnt);
+      atomicAdd((unsigned long long*)&w.pair[2 * slot + 1], (unsigned long long)cnt);
       return;
     }
   }
@@ -366,21 +425,35 @@ struct ScanAcc {
   uint64_t dsum, dxor, nh;
 };
 
+// Shared-memory state of one scan block (dynamic shared memory, see scan_smem).
+struct ScanSmem {
+  uint8_t* buf;     // kPre + chunk + kHalo + kSlack bytes; file byte p at buf[kPre + p - s]
+  uint32_t* mask;   // word-byte bits per 32-byte stripe of buf (+1 zero stripe)
+  uint32_t* ckey;   // count table: word + 1 (0 = empty)
+  uint32_t* ccnt;
+  uint16_t* olist;  // occupied count slots, in insertion order
+};
+
 // One hit of word k at file position pos: per-item shared count (spilling to
-// the global table when full), digest, optional hit list.
-__device__ __forceinline__ void count_hit(GrepWork& w, uint32_t* ckey, uint32_t* ccnt, uint32_t f, uint32_t k,
-                                          uint64_t pos, uint64_t* hits, uint64_t hit_cap, ScanAcc& acc) {
+// the global table when the probe run is exhausted), digest, optional hit list.
+__device__ __forceinline__ void count_hit(GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
+                                          uint32_t f, uint32_t k, uint64_t pos, uint64_t* hits, uint64_t hit_cap,
+                                          ScanAcc& acc) {
   uint32_t cs = (k * 2654435761u) & (kCountSlots - 1);
   bool done = false;
   for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & (kCountSlots - 1)) {
-    const uint32_t prev = atomicCAS(&ckey[cs], 0u, k + 1);
+    const uint32_t prev = atomicCAS(&S.ckey[cs], 0u, k + 1);
+    if (prev == 0) S.olist[atomicAdd(nocc, 1u)] = (uint16_t)cs;
     if (prev == 0 || prev == k + 1) {
-      atomicAdd(&ccnt[cs], 1u);
+      atomicAdd(&S.ccnt[cs], 1u);
       done = true;
       break;
     }
   }
-  if (!done) pair_add(w, f, k, 1);
+  if (!done) {  // this item's records then all go through the global table
+    pair_add(w, f, k, 1);
+    *spilled = 1;
+  }
   const uint64_t m = hit_mix(f, pos, k);
   acc.dsum += m;
   acc.dxor ^= m;
@@ -394,27 +467,85 @@ __device__ __forceinline__ void count_hit(GrepWork& w, uint32_t* ckey, uint32_t*
   }
 }
 
-__global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w, uint32_t chunk, uint64_t* hits,
-                                                   uint64_t hit_cap) {
+// One token: bytes buf[i, i + L), file position pos, 1 <= L <= 32.
+__device__ __forceinline__ void scan_token(GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
+                                           uint32_t f, uint32_t i, uint32_t L, uint64_t pos, uint64_t* hits,
+                                           uint64_t hit_cap, ScanAcc& acc) {
+  uint32_t W[12];
+  const uint4* q = (const uint4*)(S.buf + (i & ~15u));
+#pragma unroll
+  for (int j = 0; j < 3; ++j) {
+    const uint4 t = q[j];
+    W[4 * j] = t.x;
+    W[4 * j + 1] = t.y;
+    W[4 * j + 2] = t.z;
+    W[4 * j + 3] = t.w;
+  }
+  uint32_t v[8];
+  gather_token(W, i & 15u, L, v);
+  const uint64_t h = tok_hash(v, L);
+  const uint64_t want = entry_key(h, L) >> 26;
+  uint32_t slot = (uint32_t)h & w.table_mask;
+  for (;;) {
+    const uint64_t ent = __ldg((const unsigned long long*)&w.table[slot]);
+    if (ent == 0) return;
+    if (key_bits(ent) == want) {
+      const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
+      const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
+      const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
+      const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
+                         (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
+      if (same) {
+        count_hit(w, S, nocc, spilled, f, kp, pos, hits, hit_cap, acc);
+        if (ent & kDupBit) {  // the word's duplicates each count (R14)
+          for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
+            count_hit(w, S, nocc, spilled, f, d - 1, pos, hits, hit_cap, acc);
+        }
+        return;
+      }
+    }
+    slot = (slot + 1) & w.table_mask;
+  }
+}
+
+// Bits [lo, hi) of a 32-bit mask (lo, hi clamped to [0, 32]).
+__device__ __forceinline__ uint32_t bit_range(int lo, int hi) {
+  lo = min(max(lo, 0), 32);
+  hi = min(max(hi, 0), 32);
+  if (hi <= lo) return 0u;
+  const uint32_t upto_hi = hi == 32 ? 0xFFFFFFFFu : ((1u << hi) - 1u);
+  const uint32_t below_lo = lo == 32 ? 0xFFFFFFFFu : ((1u << lo) - 1u);
+  return upto_hi & ~below_lo;
+}
+
+__global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork w, uint32_t chunk, uint64_t* hits,
+                                                   uint64_t hit_cap, uint64_t* totals, uint32_t* rec,
+                                                   uint64_t rec_cap) {
   extern __shared__ __align__(16) uint8_t sm[];
-  uint8_t* buf = sm;                                                          // chunk + kPre + kHalo
-  uint32_t* ckey = (uint32_t*)(sm + ((chunk + kPre + kHalo + 15) & ~15u));    // word + 1
-  uint32_t* ccnt = ckey + kCountSlots;
-  uint16_t* starts = (uint16_t*)(ccnt + kCountSlots);                         // chunk / 2 token starts
+  const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
+  const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
+  ScanSmem S;
+  S.buf = sm;
+  S.mask = (uint32_t*)(sm + buf_bytes);
+  S.ckey = S.mask + ((nstripe_max + 1 + 3) & ~3u);
+  S.ccnt = S.ckey + kCountSlots;
+  S.olist = (uint16_t*)(S.ccnt + kCountSlots);
   __shared__ uint64_t item_s;
-  __shared__ uint32_t ntok_s;
+  __shared__ uint32_t nocc_s, spilled_s;
+  __shared__ unsigned long long rbase_s;
   const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31;
   const uint64_t nitems = w.vars[V_NITEMS];
   ScanAcc acc{0, 0, 0};
   for (uint32_t i = tid; i < kCountSlots; i += nthr) {  // dynamic smem is not cleared between launches
-    ckey[i] = 0;
-    ccnt[i] = 0;
+    S.ckey[i] = 0;
+    S.ccnt[i] = 0;
   }
   for (;;) {
     __syncthreads();
     if (tid == 0) {
       item_s = atomicAdd(&w.vars[V_NEXT], 1ull);
-      ntok_s = 0;
+      nocc_s = 0;
+      spilled_s = 0;
     }
     __syncthreads();
     const uint64_t item = item_s;
@@ -426,68 +557,60 @@ __global__ void __launch_bounds__(256) k_grep_scan(const gfs_ctx* c, GrepWork w,
     const uint64_t e = min(size, s + chunk);
     const uint64_t ws = s >= kPre ? s - kPre : 0;
     const uint64_t we = min(size, e + kHalo);
-    const int64_t r = gread(c, fd, ws, we - ws, buf);
+    // file byte p lands at buf[kPre + p - s]; (dst - ws) % 16 == 0, so gread
+    // moves the span with TMA (s is a multiple of the chunk, itself of 16)
+    const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
+    const int64_t r = gread(c, fd, ws, we - ws, S.buf + vlo);
     if (r != (int64_t)(we - ws)) {
       if (tid == 0) set_err(w, r < 0 ? r : -EIO);
       continue;
     }
-    // pass 1: compact token starts in [s, e) (file coordinates; buf[pos - ws])
-    const uint32_t n_here = (uint32_t)(e - s);
-    const uint32_t off0 = (uint32_t)(s - ws);
-    for (uint32_t q0 = 0; q0 < n_here; q0 += nthr) {
-      const uint32_t q = q0 + tid;
-      bool st = false;
-      if (q < n_here) {
-        const uint32_t bi = off0 + q;
-        st = is_word(buf[bi]) && (s + q == 0 || !is_word(buf[bi - 1]));
+    // pass 1: word-byte bits per 32-byte stripe; bytes outside [vlo, vhi) are non-word
+    const uint32_t nstripe = (vhi + 31) / 32;
+    for (uint32_t j = tid; j < nstripe; j += nthr)
+      S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
+    if (tid == 0) S.mask[nstripe] = 0;
+    __syncthreads();
+    // pass 2: tokens starting in [s, e) = buf[kPre, kPre + e - s), by stripe
+    const uint32_t olo = kPre, ohi = kPre + (uint32_t)(e - s);
+    for (uint32_t j = olo / 32 + tid; j <= (ohi - 1) / 32; j += nthr) {
+      const uint32_t m = S.mask[j];
+      const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
+      uint32_t st = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
+      if (!st) continue;
+      const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | m;
+      while (st) {
+        const uint32_t b = __ffs(st) - 1;
+        st &= st - 1;
+        const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
+        if (L > 32) continue;                          // no dictionary word is longer (R12)
+        const uint32_t i = 32 * j + b;
+        scan_token(w, S, &nocc_s, &spilled_s, f, i, L, s + i - kPre, hits, hit_cap, acc);
       }
-      const uint32_t bal = __ballot_sync(0xFFFFFFFFu, st);
-      uint32_t base = 0;
-      if (lane == 0 && bal) base = atomicAdd(&ntok_s, __popc(bal));
-      base = __shfl_sync(0xFFFFFFFFu, base, 0);
-      if (st) starts[base + __popc(bal & ((1u << lane) - 1))] = (uint16_t)q;
     }
     __syncthreads();
-    const uint32_t ntok = ntok_s;
-    // pass 2: whole tokens per thread
-    for (uint32_t t = tid; t < ntok; t += nthr) {
-      const uint32_t q = starts[t];
-      const uint64_t pos = s + q;
-      const uint32_t bi = off0 + q;
-      uint32_t L = 1;
-      while (L <= 32 && pos + L < size && is_word(buf[bi + L])) ++L;
-      if (L > 32) continue;  // tokens longer than any dictionary word never match
-      const uint64_t h = tok_hash(buf + bi, L);
-      const uint64_t want = entry_key(h, L) >> 26;
-      uint32_t slot = (uint32_t)h & w.table_mask;
-      for (;;) {
-        const uint64_t ent = __ldg((const unsigned long long*)&w.table[slot]);
-        if (ent == 0) break;
-        if (key_bits(ent) == want) {
-          const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
-          const uint8_t* tw = w.dict + (size_t)kp * 32;
-          bool same = true;
-          for (uint32_t i = 0; i < L; ++i) same &= __ldg(tw + i) == buf[bi + i];
-          if (same) {
-            count_hit(w, ckey, ccnt, f, kp, pos, hits, hit_cap, acc);
-            if (ent & kDupBit) {  // the word's duplicates each count (R14)
-              for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
-                count_hit(w, ckey, ccnt, f, d - 1, pos, hits, hit_cap, acc);
-            }
-            break;
-          }
+    // flush: a whole-file item with no spill owns its records; otherwise merge
+    const uint32_t nocc = nocc_s;
+    const bool direct = s == 0 && e == size && !spilled_s && rec;
+    if (direct && tid == 0 && nocc) rbase_s = atomicAdd(&w.vars[V_NREC], (unsigned long long)nocc);
+    __syncthreads();
+    for (uint32_t q = tid; q < nocc; q += nthr) {
+      const uint32_t cs = S.olist[q];
+      const uint32_t k = S.ckey[cs] - 1, cnt = S.ccnt[cs];
+      S.ckey[cs] = 0;
+      S.ccnt[cs] = 0;
+      if (direct) {
+        atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
+        const uint64_t idx = rbase_s + q;
+        if (idx < rec_cap) {
+          rec[3 * idx] = f;
+          rec[3 * idx + 1] = k;
+          rec[3 * idx + 2] = cnt;
+        } else {
+          set_err(w, -ENOSPC);
         }
-        slot = (slot + 1) & w.table_mask;
-      }
-    }
-    __syncthreads();
-    // flush this item's counts into the (file, word) table
-    for (uint32_t i = tid; i < kCountSlots; i += nthr) {
-      const uint32_t kk = ckey[i];
-      if (kk) {
-        pair_add(w, f, kk - 1, ccnt[i]);
-        ckey[i] = 0;
-        ccnt[i] = 0;
+      } else {
+        pair_add(w, f, k, cnt);
       }
     }
   }
@@ -519,14 +642,14 @@ __global__ void k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap, uint
   const uint64_t n = w.pair_mask + 1;
   for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x; i0 < n; i0 += stride) {
     const uint64_t i = i0 + threadIdx.x;
-    const uint64_t key = i < n ? w.pair_key[i] : kPairEmpty;
+    const uint64_t key = i < n ? w.pair[2 * i] : kPairEmpty;
     const bool v = key != kPairEmpty;
     const uint32_t bal = __ballot_sync(0xFFFFFFFFu, v);
     unsigned long long base = 0;
     if (lane == 0 && bal) base = atomicAdd(&w.vars[V_NREC], (unsigned long long)__popc(bal));
     base = __shfl_sync(0xFFFFFFFFu, base, 0);
     if (v) {
-      const uint64_t cnt = w.pair_cnt[i];
+      const uint64_t cnt = w.pair[2 * i + 1];
       const uint32_t k = (uint32_t)key;
       atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
       const uint64_t idx = base + __popc(bal & ((1u << lane) - 1));
@@ -534,6 +657,8 @@ __global__ void k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap, uint
         rec[3 * idx] = (uint32_t)(key >> 32);
         rec[3 * idx + 1] = k;
         rec[3 * idx + 2] = (uint32_t)cnt;
+      } else if (rec) {
+        set_err(w, -ENOSPC);
       }
     }
   }
@@ -543,8 +668,8 @@ __global__ void k_grep_init(GrepWork w, uint32_t max_words) {
   const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
   const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
   for (uint64_t i = t; i <= w.pair_mask; i += stride) {
-    w.pair_key[i] = kPairEmpty;
-    w.pair_cnt[i] = 0;
+    w.pair[2 * i] = kPairEmpty;
+    w.pair[2 * i + 1] = 0;
   }
   for (uint64_t i = t; i <= w.table_mask; i += stride) w.table[i] = 0;
   for (uint64_t i = t; i < max_words; i += stride) {
@@ -599,8 +724,8 @@ Layout layout(const gfs_grep_params* p) {
       (uint64_t)p->max_files * 8,                          // size
       ((uint64_t)p->max_files + 1) * 8,                    // item_base
       L.max_items * 4,                                     // item_file
-      pcap * 8,                                            // pair_key
-      pcap * 8,                                            // pair_cnt
+      pcap * 16,                                           // pair
+      0,                                                   // (unused)
       V_NVARS * 8,                                         // vars
   };
   uint64_t o = 0;
@@ -613,7 +738,9 @@ Layout layout(const gfs_grep_params* p) {
 }
 
 uint32_t scan_smem(uint32_t chunk) {
-  return ((chunk + kPre + kHalo + 15) & ~15u) + 2 * kCountSlots * 4 + (chunk / 2 + 16) * 2;
+  const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
+  const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
+  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * kCountSlots * 4 + kCountSlots * 2;
 }
 
 }  // namespace
@@ -644,8 +771,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   w.item_base = (uint64_t*)(base + L.off[9]);
   w.item_file = (uint32_t*)(base + L.off[10]);
   w.max_items = L.max_items;
-  w.pair_key = (uint64_t*)(base + L.off[11]);
-  w.pair_cnt = (uint64_t*)(base + L.off[12]);
+  w.pair = (uint64_t*)(base + L.off[11]);
   w.pair_mask = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap) - 1;
   w.vars = (unsigned long long*)(base + L.off[13]);
 
@@ -697,24 +823,37 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
             (long long)v[V_ERR], v[V_NFILES], v[V_NWORDS], v[V_NITEMS], v[V_BYTES]);
     ts_prev = ts;
   };
-  const uint64_t lb = p->list_cap / kListChunk + 1;
+  const uint64_t lb = p->list_cap / kListChunk + 1, lr = p->list_cap / kListRead + 1;
   const uint32_t list_blocks = (uint32_t)(lb < 1024 ? lb : 1024);
+  // one opener per 64 KiB piece: a block that opens the list after all others
+  // closed it would re-validate it with the host (close-to-open)
+  const uint32_t read_blocks = (uint32_t)(lr < 1024 ? lr : 1024);
   k_grep_init<<<1024, 256, 0, s>>>(w, p->max_words);
   k_grep_dict<<<64, 256, 0, s>>>(c, d_str, w, p->max_words);
   stage("dict");
-  k_grep_list_read<<<list_blocks, 256, 0, s>>>(c, d_str + kMaxPath, w, p->list_cap);
+  k_grep_list_read<<<read_blocks, 256, 0, s>>>(c, d_str + kMaxPath, w, p->list_cap);
   k_grep_list_count<<<list_blocks, 256, 0, s>>>(w);
   k_grep_list_scan<<<1, 32, 0, s>>>(w, p->max_files);
   k_grep_list_emit<<<list_blocks, 256, 0, s>>>(w, d_str + 2 * kMaxPath, (uint32_t)dl, p->max_files);
   stage("list");
-  k_grep_open<<<p->grid, 128, 0, s>>>(c, w, p->chunk);
+  // gopen is block-collective with one leader thread: many one-warp blocks
+  // keep more opens in flight (host RPCs when cold, L2 round trips when warm)
+  int dev = 0, nsm = 148;
+  cudaGetDevice(&dev);
+  cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
+  k_grep_open<<<nsm * 16, 32, 0, s>>>(c, w, p->chunk);
   stage("open");
   k_grep_plan<<<1, 1024, 0, s>>>(w);
   k_grep_items<<<256, 256, 0, s>>>(w);
-  k_grep_scan<<<p->grid, p->block, smem, s>>>(c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0);
-  stage("scan");
-  if (!p->keep_open) k_grep_close<<<p->grid, 32, 0, s>>>(c, w);
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
+  // persistent scan grid: every resident block slot once (p->grid caps it)
+  int occ = 1;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_scan, (int)p->block, smem);
+  const uint32_t scan_grid = (uint32_t)(occ > 0 ? occ : 1) * (uint32_t)nsm;
+  k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
+      c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
+  stage("scan");
+  if (!p->keep_open) k_grep_close<<<nsm * 16, 32, 0, s>>>(c, w);
   k_grep_compact<<<1024, 256, 0, s>>>(w, d_rec, d_rec ? rec_cap : 0, d_totals);
   k_grep_summary<<<1, 32, 0, s>>>(w, d_summary);
   stage("done");

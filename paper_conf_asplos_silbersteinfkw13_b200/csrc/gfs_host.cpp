@@ -229,7 +229,7 @@ int cuda_err(cudaError_t e) {
     }                                 \
   } while (0)
 
-uint32_t alloc_hfid(gfs_handle* h, HostFile f) {
+uint32_t alloc_hfid(gfs_handle* h, HostFile&& f, uint32_t* gen_out) {
   std::lock_guard<std::mutex> g(h->fd_mu);
   f.live = true;
   uint32_t id;
@@ -237,12 +237,13 @@ uint32_t alloc_hfid(gfs_handle* h, HostFile f) {
     id = h->free_hfids.back();
     h->free_hfids.pop_back();
     f.gen = h->files[id].gen;
-    h->files[id] = f;
+    h->files[id] = std::move(f);
   } else {
     f.gen = 0;
-    h->files.push_back(f);
+    h->files.push_back(std::move(f));
     id = (uint32_t)(h->files.size() - 1);
   }
+  *gen_out = h->files[id].gen;
   return id;
 }
 
@@ -456,11 +457,10 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
     f.dev = st.st_dev;
     f.ino = st.st_ino;
     f.size = (uint64_t)st.st_size;
-    f.path = path;
-    hfid = alloc_hfid(h, f);
-    HostFile m;
-    if (hfid_meta(h, hfid, &m)) w_cache(w, hfid, fd, m.gen);
-    else ::close(fd);
+    f.path = std::move(path);
+    uint32_t gen;
+    hfid = alloc_hfid(h, std::move(f), &gen);
+    w_cache(w, hfid, fd, gen);
   }
   rs->size = (int64_t)st.st_size;
   rs->version = h->vt.get(st.st_dev, st.st_ino);
@@ -711,6 +711,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   gfs_ctx& c = h->h;
   const uint32_t R = cfg->ring_slots;
   const uint32_t MF = cfg->max_files;
+  h->files.reserve(MF);  // host metadata grows under fd_mu: no reallocation in the OPEN path
   const uint32_t max_nodes = cfg->max_nodes ? cfg->max_nodes : (MF * 2u + 65536u);
   const size_t ctr_bytes = (size_t)GFS_C_NCOUNTERS * GFS_CTR_SHARDS * sizeof(unsigned long long);
   uint32_t slots = cfg->staging_slots;

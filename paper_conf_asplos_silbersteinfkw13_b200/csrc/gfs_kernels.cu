@@ -111,13 +111,18 @@ __global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint
       } else {
         r = 0;
       }
-    } else if (len[i] > smem_bytes) {
-      r = -EINVAL;  // destination would overflow the shared buffer
     } else {
-      r = gread(c, fd, off[i], len[i], smem);
-      if (r > 0)
-        for (int64_t k = tid; k < r; k += blockDim.x) dst[dstoff[i] + k] = smem[k];
-      __syncthreads();
+      // mode 2: shared buffer at its aligned base; mode 3: at off % 16, so the
+      // destination is co-aligned with the file offset (TMA middle + edges)
+      const uint32_t sh = mode == 3 ? (uint32_t)(off[i] & 15) : 0u;
+      if (len[i] + sh > smem_bytes) {
+        r = -EINVAL;  // destination would overflow the shared buffer
+      } else {
+        r = gread(c, fd, off[i], len[i], smem + sh);
+        if (r > 0)
+          for (int64_t k = tid; k < r; k += blockDim.x) dst[dstoff[i] + k] = smem[sh + k];
+        __syncthreads();
+      }
     }
     if (tid == 0) ret[i] = r;
   }
@@ -298,13 +303,13 @@ extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s) {
 GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
                           const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
                           int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes) {
-  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || mode > 2) return -EINVAL;
+  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || mode > 3) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
   const char* dp = stage_path(path, s);
   if (!dp) return -ENAMETOOLONG;
-  if (mode == 2 && smem_bytes > 48 * 1024)
+  if (mode >= 2 && smem_bytes > 48 * 1024)
     cudaFuncSetAttribute(k_gread_calls, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem_bytes);
-  k_gread_calls<<<grid, block, mode == 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,
+  k_gread_calls<<<grid, block, mode >= 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,
                                                                 d_dstoff, d_dst, d_ret, smem_bytes);
   return launch_err(cudaGetLastError());
 }

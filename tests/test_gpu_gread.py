@@ -98,6 +98,22 @@ def test_gread_into_shared_memory(g, shmdir):
     check_calls(path, size, offs[ok], lens[ok], ret[ok], dst, dstoff[ok])
 
 
+@pytest.mark.parametrize("P", [4096, 65536])
+def test_gread_into_shared_memory_coaligned(g, shmdir, P):
+    """Destination at off % 16 in shared memory: the TMA path moves the aligned
+    middle of every page span, warp 0 the unaligned head and tail bytes."""
+    size = 40 * P + 777
+    path = gen.splitmix_file(os.path.join(shmdir, "sc.bin"), size, seed=11)
+    offs, lens = gen.random_calls(9, 400, size, 3 * P, page_size=P)
+    lens = np.minimum(lens, 32768 - 16)
+    lens[:8] = [0, 1, 15, 16, 17, 31, 33, 4095]
+    offs[:8] = [3, 1, 7, size - 5, P - 3, 2 * P - 16, 13, size - 100]
+    offs[8], lens[8] = P - 1, 2  # one byte on each side of a page boundary
+    with _fs(g, cache_bytes=24 * P, page_size=P) as fs:  # < file: misses and evictions too
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, mode=3, grid=2, smem=32768)
+    check_calls(path, size, offs, lens, ret, dst, dstoff)
+
+
 @pytest.mark.parametrize("locked", [0, 1])
 def test_locked_traversal_same_bytes(g, shmdir, locked):
     P = 4096

@@ -10,7 +10,7 @@ c = gen.c4_corpus(f"/dev/shm/gfs_bench_c4_{nf}_{mib}", seed=4, nfiles=nf, total_
 with g.GpuFS(cache_bytes=4 << 30, page_size=64 << 10, daemon_threads=12, max_files=1 << 16) as fs:
     for phase in ("cold", "warm"):
         t = time.time()
-        out = fs.grep(c["dict"], c["list"], keep_open=True, pair_cap=1 << 24)
+        out = fs.grep(c["dict"], c["list"], keep_open=True, rec_cap=1 << 24)
         print(phase, f"{(time.time()-t)*1e3:.1f} ms", out["summary"], flush=True)
     print(fs.stats())
     print(fs.host_stats())
