@@ -1063,12 +1063,52 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
 }
 
 // ------------------------------------------------------------------ file table
-__device__ __forceinline__ uint64_t path_hash(const char* p, uint32_t n) {
-  uint64_t h = 1469598103934665603ull;
-  for (uint32_t i = 0; i < n; ++i) h = (h ^ (uint8_t)p[i]) * 1099511628211ull;
-  return h;
+// Path hash: an order-sensitive SUM of per-(position, byte) mixes, so a warp
+// can hash a path in parallel (lane l takes bytes l, l+32, ...).
+__device__ __forceinline__ uint64_t path_term(uint32_t i, uint32_t b) {
+  uint64_t z = (((uint64_t)i << 8) | b) * 0x9E3779B97F4A7C15ull;
+  z = (z ^ (z >> 29)) * 0xBF58476D1CE4E5B9ull;
+  return z ^ (z >> 32);
 }
-
+__device__ __forceinline__ uint64_t path_final(uint64_t sum, uint32_t n) {
+  uint64_t z = sum ^ ((uint64_t)n * 0x94D049BB133111EBull);
+  z = (z ^ (z >> 31)) * 0xBF58476D1CE4E5B9ull;
+  return z ^ (z >> 29);
+}
+// Length (GFS_MAX_PATH if no NUL within it) and hash of `p`, by one thread.
+__device__ __forceinline__ uint32_t path_len_hash(const char* p, uint64_t* h) {
+  uint32_t n = 0;
+  uint64_t sum = 0;
+  while (n < GFS_MAX_PATH && p[n]) {
+    sum += path_term(n, (uint8_t)p[n]);
+    ++n;
+  }
+  *h = path_final(sum, n);
+  return n;
+}
+// The same, by a full warp: one aligned 32-byte window per step (coalesced,
+// never crosses a page, so no read faults past the NUL), one ballot per step.
+__device__ __forceinline__ uint32_t path_len_hash_warp(const char* p, uint64_t* h) {
+  const int lane = block_tid() & 31;
+  const int off0 = (int)((uintptr_t)p & 31);
+  const unsigned char* a = (const unsigned char*)((uintptr_t)p & ~(uintptr_t)31);
+  uint64_t sum = 0;
+  uint32_t n = GFS_MAX_PATH;
+  for (int base = 0; base < (int)GFS_MAX_PATH + off0; base += 32) {
+    const int i = base + lane - off0;  // index in the path; < 0: before it
+    const uint32_t b = (i >= 0 && i < (int)GFS_MAX_PATH) ? a[base + lane] : 1u;
+    const uint32_t z = __ballot_sync(0xFFFFFFFFu, b == 0);
+    const int lim = z ? base + (__ffs(z) - 1) - off0 : (int)GFS_MAX_PATH;  // bytes before the NUL
+    if (i >= 0 && i < lim) sum += path_term((uint32_t)i, b);
+    if (z) {
+      n = (uint32_t)lim;
+      break;
+    }
+  }
+  for (int o = 16; o; o >>= 1) sum += __shfl_xor_sync(0xFFFFFFFFu, sum, o);
+  *h = path_final(sum, n);
+  return n;
+}
 __device__ __forceinline__ bool snap_fd(const gfs_ctx* c, int fd, FileSnap* s) {
   if (fd < 0 || (uint32_t)fd >= c->max_files) return false;
   const gfs_file* e = c->files + fd;
@@ -1164,9 +1204,21 @@ __device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uin
 __device__ __forceinline__ bool same_path(const gfs_ctx* c, const gfs_file* e, uint32_t fdx, const char* path,
                                           uint32_t n, uint64_t h) {
   if (ld_rlx64(&e->path_hash) != h || ld_rlx(&e->path_len) != n) return false;
-  const volatile char* sp = c->paths + (size_t)fdx * GFS_MAX_PATH;
+  const char* sp = c->paths + (size_t)fdx * GFS_MAX_PATH;  // 1 KiB aligned
+  if ((((uintptr_t)path) & 7) == 0) {
+    // 8-byte words, no early exit (the loads pipeline); an aligned word never
+    // crosses a page, so reading the caller's word holding the NUL is safe
+    const uint32_t nw = (n + 7) / 8;
+    uint64_t diff = 0;
+    for (uint32_t k = 0; k < nw; ++k) {
+      uint64_t x = __ldcg((const unsigned long long*)sp + k) ^ ((const unsigned long long*)path)[k];
+      if (k == nw - 1 && (n & 7)) x &= (1ull << (8 * (n & 7))) - 1;
+      diff |= x;
+    }
+    return diff == 0;
+  }
   for (uint32_t i = 0; i < n; ++i)
-    if (sp[i] != path[i]) return false;
+    if (__ldcg((const unsigned char*)sp + i) != (unsigned char)path[i]) return false;
   return true;
 }
 
@@ -1214,17 +1266,16 @@ struct Prefetch {
 };
 
 // gopen body, run by one thread.
-__device__ int open_leader(const gfs_ctx* c, const char* path, int flags_in, Prefetch* pf) {
+// `n`, `h`: the path's length and hash (path_len_hash*).
+__device__ int open_leader(const gfs_ctx* c, const char* path, uint32_t n, uint64_t h, int flags_in,
+                           Prefetch* pf) {
   pf->frame = -1;
   pf->stage = -1;
   const bool want_pf = (flags_in & (int)GFS_O_PREFETCH) != 0;
   const int flags = flags_in & ~(int)GFS_O_PREFETCH;
   if (flags != (int)GFS_O_RDONLY && flags != (int)GFS_O_GWRONCE) return -EINVAL;
-  uint32_t n = 0;
-  while (n < GFS_MAX_PATH && path[n]) ++n;
   if (n == 0) return -ENOENT;
   if (n >= GFS_MAX_PATH) return -ENAMETOOLONG;
-  const uint64_t h = path_hash(path, n);
   const uint32_t mask = c->max_files - 1;
   uint32_t i = (uint32_t)h & mask;
   uint32_t probes = 0;
@@ -1391,9 +1442,16 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
   Scratch& sc = detail::scratch();
   const int tid = detail::block_tid();
   __syncthreads();
+  uint64_t ph = 0;
+  uint32_t pn = 0;
+  if (detail::block_nthr() >= 32) {  // warp 0 measures and hashes the path together
+    if (tid < 32) pn = detail::path_len_hash_warp(path, &ph);
+  } else if (tid == 0) {
+    pn = detail::path_len_hash(path, &ph);
+  }
   if (tid == 0) {
     detail::Prefetch pf;
-    const int fd = detail::open_leader(c, path, flags, &pf);
+    const int fd = detail::open_leader(c, path, pn, ph, flags, &pf);
     sc.ret = fd;
     sc.frame[0] = pf.frame;
     sc.stage[0] = pf.stage;

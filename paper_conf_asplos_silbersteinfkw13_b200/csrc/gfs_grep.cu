@@ -81,7 +81,7 @@ struct GrepWork {
   unsigned long long* vars;  // see V_*
 };
 enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS, V_DSUM, V_DXOR, V_NLISTED,
-       V_NEXTF, V_LISTSZ, V_NVARS };
+       V_NEXTF, V_LISTSZ, V_HOLD_DICT, V_HOLD_LIST, V_NVARS };
 
 __device__ __forceinline__ bool is_word(uint32_t ch) {
   return (ch - 'a' < 26u) || (ch - 'A' < 26u) || (ch - '0' < 10u) || ch == '_';
@@ -161,6 +161,26 @@ __device__ __forceinline__ uint64_t hit_mix(uint64_t f, uint64_t off, uint64_t k
 
 __device__ __forceinline__ void set_err(GrepWork& w, long long e) { atomicMin((long long*)&w.vars[V_ERR], e); }
 
+// --------------------------------------------------------------- hold
+// One block opens the dictionary and the list before the blocks that read
+// them and closes them after the run: the many short gopen/gclose pairs of
+// the reading blocks then never drop the count to zero, which would make the
+// next opener re-validate the file with the host (close-to-open).
+__global__ void k_grep_hold(const gfs_ctx* c, const char* dict_path, const char* list_path, GrepWork w, int release) {
+  if (!release) {
+    const int a = gopen(c, dict_path, GFS_O_RDONLY);
+    const int b = gopen(c, list_path, GFS_O_RDONLY);
+    if (threadIdx.x == 0) {
+      w.vars[V_HOLD_DICT] = (unsigned long long)(long long)a;
+      w.vars[V_HOLD_LIST] = (unsigned long long)(long long)b;
+    }
+  } else {
+    const int a = (int)(long long)w.vars[V_HOLD_DICT], b = (int)(long long)w.vars[V_HOLD_LIST];
+    if (a >= 0) gclose(c, a);
+    if (b >= 0) gclose(c, b);
+  }
+}
+
 // --------------------------------------------------------------- dictionary
 __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w, uint32_t max_words) {
   const int tid = threadIdx.x;
@@ -204,7 +224,9 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
         for (int j = 0; j < 8; ++j) v[j] = ((const uint32_t*)s)[j];
         const uint64_t h = tok_hash(v, n);
         const uint64_t ent = entry_key(h, n) | (k + 1);
-        uint32_t slot = (uint32_t)h & w.table_mask;
+        // linear probing from the start of the hash's 4-entry (32-byte) bucket:
+        // lookups read a whole bucket per step (scan_token)
+        uint32_t slot = (uint32_t)h & w.table_mask & ~3u;
         for (uint32_t probe = 0; probe <= w.table_mask; ++probe, slot = (slot + 1) & w.table_mask) {
           unsigned long long cur = atomicCAS((unsigned long long*)&w.table[slot], 0ull, (unsigned long long)ent);
           if (cur == 0) break;
@@ -485,26 +507,36 @@ __device__ __forceinline__ void scan_token(GrepWork& w, const ScanSmem& S, uint3
   gather_token(W, i & 15u, L, v);
   const uint64_t h = tok_hash(v, L);
   const uint64_t want = entry_key(h, L) >> 26;
-  uint32_t slot = (uint32_t)h & w.table_mask;
+  // One 32-byte bucket (4 entries) per step; insertion filled the first empty
+  // slot in the same order, so an empty slot ends the search.
+  uint32_t b = (uint32_t)h & w.table_mask & ~3u;
   for (;;) {
-    const uint64_t ent = __ldg((const unsigned long long*)&w.table[slot]);
-    if (ent == 0) return;
-    if (key_bits(ent) == want) {
-      const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
-      const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
-      const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
-      const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
-                         (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
-      if (same) {
-        count_hit(w, S, nocc, spilled, f, kp, pos, hits, hit_cap, acc);
-        if (ent & kDupBit) {  // the word's duplicates each count (R14)
-          for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
-            count_hit(w, S, nocc, spilled, f, d - 1, pos, hits, hit_cap, acc);
+    const uint4* bp = (const uint4*)&w.table[b];
+    const uint4 e01 = __ldg(bp), e23 = __ldg(bp + 1);
+    const uint64_t ent[4] = {((uint64_t)e01.y << 32) | e01.x, ((uint64_t)e01.w << 32) | e01.z,
+                             ((uint64_t)e23.y << 32) | e23.x, ((uint64_t)e23.w << 32) | e23.z};
+    bool empty = false;
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      empty |= ent[q] == 0;
+      if (ent[q] != 0 && key_bits(ent[q]) == want) {
+        const uint32_t kp = (uint32_t)(ent[q] & ((1u << 26) - 1)) - 1;
+        const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
+        const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
+        const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
+                           (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
+        if (same) {
+          count_hit(w, S, nocc, spilled, f, kp, pos, hits, hit_cap, acc);
+          if (ent[q] & kDupBit) {  // the word's duplicates each count (R14)
+            for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
+              count_hit(w, S, nocc, spilled, f, d - 1, pos, hits, hit_cap, acc);
+          }
+          return;
         }
-        return;
       }
     }
-    slot = (slot + 1) & w.table_mask;
+    if (empty) return;
+    b = (b + 4) & w.table_mask;
   }
 }
 
@@ -522,6 +554,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
                                                    uint64_t hit_cap, uint64_t* totals, uint32_t* rec,
                                                    uint64_t rec_cap) {
   extern __shared__ __align__(16) uint8_t sm[];
+  const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31, wid = tid >> 5;
   const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
   const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
   ScanSmem S;
@@ -530,39 +563,58 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
   S.ckey = S.mask + ((nstripe_max + 1 + 3) & ~3u);
   S.ccnt = S.ckey + kCountSlots;
   S.olist = (uint16_t*)(S.ccnt + kCountSlots);
-  __shared__ uint64_t item_s;
+  uint16_t* tok = S.olist + kCountSlots;  // token starts of one round: <= 32 per thread
+  const uint32_t round_stripes = 2u * (uint32_t)nthr;
+  __shared__ uint64_t nxt_item, nxt_size, nxt_base;
+  __shared__ uint32_t nxt_f;
+  __shared__ int32_t nxt_fd;
   __shared__ uint32_t nocc_s, spilled_s;
+  __shared__ uint32_t warp_tot[32];
   __shared__ unsigned long long rbase_s;
-  const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31;
   const uint64_t nitems = w.vars[V_NITEMS];
   ScanAcc acc{0, 0, 0};
+  // tid 0 claims the next item and loads its file fields while the block
+  // works on the current one (three dependent L2 round trips off the path)
+  auto prefetch = [&]() {
+    const uint64_t it = atomicAdd(&w.vars[V_NEXT], 1ull);
+    nxt_item = it;
+    if (it < nitems) {
+      const uint32_t f = w.item_file[it];
+      nxt_f = f;
+      nxt_fd = w.fd[f];
+      nxt_size = w.size[f];
+      nxt_base = w.item_base[f];
+    }
+  };
   for (uint32_t i = tid; i < kCountSlots; i += nthr) {  // dynamic smem is not cleared between launches
     S.ckey[i] = 0;
     S.ccnt[i] = 0;
   }
+  if (tid == 0) prefetch();
   for (;;) {
     __syncthreads();
+    const uint64_t item = nxt_item;
+    if (item >= nitems) break;
+    const uint32_t f = nxt_f;
+    const int fd = nxt_fd;
+    const uint64_t size = nxt_size;
+    const uint64_t s = (item - nxt_base) * chunk;
     if (tid == 0) {
-      item_s = atomicAdd(&w.vars[V_NEXT], 1ull);
       nocc_s = 0;
       spilled_s = 0;
     }
-    __syncthreads();
-    const uint64_t item = item_s;
-    if (item >= nitems) break;
-    const uint32_t f = w.item_file[item];
-    const int fd = w.fd[f];
-    const uint64_t size = w.size[f];
-    const uint64_t s = (item - w.item_base[f]) * chunk;
     const uint64_t e = min(size, s + chunk);
     const uint64_t ws = s >= kPre ? s - kPre : 0;
     const uint64_t we = min(size, e + kHalo);
     // file byte p lands at buf[kPre + p - s]; (dst - ws) % 16 == 0, so gread
     // moves the span with TMA (s is a multiple of the chunk, itself of 16)
     const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
-    const int64_t r = gread(c, fd, ws, we - ws, S.buf + vlo);
+    const int64_t r = gread(c, fd, ws, we - ws, S.buf + vlo);  // starts with a barrier
     if (r != (int64_t)(we - ws)) {
-      if (tid == 0) set_err(w, r < 0 ? r : -EIO);
+      if (tid == 0) {
+        set_err(w, r < 0 ? r : -EIO);
+        prefetch();
+      }
       continue;
     }
     // pass 1: word-byte bits per 32-byte stripe; bytes outside [vlo, vhi) are non-word
@@ -571,24 +623,54 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
       S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
     if (tid == 0) S.mask[nstripe] = 0;
     __syncthreads();
-    // pass 2: tokens starting in [s, e) = buf[kPre, kPre + e - s), by stripe
+    if (tid == 0) prefetch();  // next item's fields, overlapping pass 2
+    // pass 2, by rounds of 2 stripes per thread: the starts of tokens in
+    // [s, e) = buf[kPre, kPre + e - s) are compacted into `tok`, then every
+    // thread takes every nthr-th token (balanced whatever the text layout)
     const uint32_t olo = kPre, ohi = kPre + (uint32_t)(e - s);
-    for (uint32_t j = olo / 32 + tid; j <= (ohi - 1) / 32; j += nthr) {
-      const uint32_t m = S.mask[j];
-      const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
-      uint32_t st = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
-      if (!st) continue;
-      const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | m;
-      while (st) {
-        const uint32_t b = __ffs(st) - 1;
-        st &= st - 1;
-        const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
-        if (L > 32) continue;                          // no dictionary word is longer (R12)
-        const uint32_t i = 32 * j + b;
-        scan_token(w, S, &nocc_s, &spilled_s, f, i, L, s + i - kPre, hits, hit_cap, acc);
+    const uint32_t jlo = olo / 32, jhi = (ohi - 1) / 32;
+    for (uint32_t r0 = jlo; r0 <= jhi; r0 += round_stripes) {
+      uint32_t st[2];
+      uint32_t cnt = 0;
+#pragma unroll
+      for (int q = 0; q < 2; ++q) {
+        const uint32_t j = r0 + 2 * (uint32_t)tid + q;
+        st[q] = 0;
+        if (j <= jhi) {
+          const uint32_t m = S.mask[j];
+          const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
+          st[q] = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
+        }
+        cnt += __popc(st[q]);
       }
+      uint32_t incl = cnt;
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+        if (lane >= o) incl += t;
+      }
+      if (lane == 31) warp_tot[wid] = incl;
+      __syncthreads();
+      uint32_t off = incl - cnt, total = 0;
+      for (int q = 0; q < (nthr >> 5); ++q) {
+        const uint32_t t = warp_tot[q];
+        off += q < wid ? t : 0u;
+        total += t;
+      }
+#pragma unroll
+      for (int q = 0; q < 2; ++q) {
+        const uint32_t jb = 32 * (r0 + 2 * (uint32_t)tid + q);
+        for (uint32_t x = st[q]; x; x &= x - 1) tok[off++] = (uint16_t)(jb + __ffs(x) - 1);
+      }
+      __syncthreads();
+      for (uint32_t q = tid; q < total; q += nthr) {
+        const uint32_t i = tok[q], j = i >> 5, b = i & 31;
+        const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | S.mask[j];
+        const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
+        if (L <= 32)                                   // no dictionary word is longer (R12)
+          scan_token(w, S, &nocc_s, &spilled_s, f, i, L, s + i - kPre, hits, hit_cap, acc);
+      }
+      __syncthreads();  // tok and warp_tot are reused by the next round
     }
-    __syncthreads();
     // flush: a whole-file item with no spill owns its records; otherwise merge
     const uint32_t nocc = nocc_s;
     const bool direct = s == 0 && e == size && !spilled_s && rec;
@@ -635,32 +717,58 @@ __global__ void k_grep_close(const gfs_ctx* c, GrepWork w) {
   }
 }
 
-// unique records from the (file, word) table + word totals (warp-aggregated output index)
-__global__ void k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap, uint64_t* totals) {
-  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-  const int lane = threadIdx.x & 31;
-  const uint64_t n = w.pair_mask + 1;
-  for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x; i0 < n; i0 += stride) {
-    const uint64_t i = i0 + threadIdx.x;
-    const uint64_t key = i < n ? w.pair[2 * i] : kPairEmpty;
-    const bool v = key != kPairEmpty;
-    const uint32_t bal = __ballot_sync(0xFFFFFFFFu, v);
-    unsigned long long base = 0;
-    if (lane == 0 && bal) base = atomicAdd(&w.vars[V_NREC], (unsigned long long)__popc(bal));
-    base = __shfl_sync(0xFFFFFFFFu, base, 0);
-    if (v) {
-      const uint64_t cnt = w.pair[2 * i + 1];
-      const uint32_t k = (uint32_t)key;
-      atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
-      const uint64_t idx = base + __popc(bal & ((1u << lane) - 1));
+// Unique records from the (file, word) table + word totals. A block takes
+// 1024 consecutive slots (4 per thread, 64 contiguous bytes), scans the valid
+// counts and reserves its output range with one atomic.
+__global__ void __launch_bounds__(256) k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap,
+                                                      uint64_t* totals) {
+  __shared__ uint32_t warp_tot[8];
+  __shared__ unsigned long long base_s;
+  const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
+  const uint64_t n = w.pair_mask + 1;  // a power of two >= 1024
+  for (uint64_t blk = blockIdx.x; blk * 1024 < n; blk += gridDim.x) {
+    const uint64_t i0 = blk * 1024 + (uint64_t)tid * 4;
+    const uint4* src = (const uint4*)(w.pair + 2 * i0);
+    uint64_t key[4], cnt[4];
+    uint32_t nv = 0;
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      const uint4 v = src[q];
+      key[q] = ((uint64_t)v.y << 32) | v.x;
+      cnt[q] = ((uint64_t)v.w << 32) | v.z;
+      nv += key[q] != kPairEmpty;
+    }
+    uint32_t incl = nv;  // inclusive scan in the warp, then across warps
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+      if (lane >= o) incl += t;
+    }
+    if (lane == 31) warp_tot[wid] = incl;
+    __syncthreads();
+    uint32_t before = 0, all = 0;
+    for (int q = 0; q < 8; ++q) {
+      const uint32_t t = warp_tot[q];
+      before += q < wid ? t : 0u;
+      all += t;
+    }
+    if (tid == 0) base_s = all ? atomicAdd(&w.vars[V_NREC], (unsigned long long)all) : 0ull;
+    __syncthreads();
+    uint64_t idx = base_s + before + incl - nv;
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      if (key[q] == kPairEmpty) continue;
+      const uint32_t k = (uint32_t)key[q];
+      atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt[q]);
       if (idx < rec_cap) {
-        rec[3 * idx] = (uint32_t)(key >> 32);
+        rec[3 * idx] = (uint32_t)(key[q] >> 32);
         rec[3 * idx + 1] = k;
-        rec[3 * idx + 2] = (uint32_t)cnt;
+        rec[3 * idx + 2] = (uint32_t)cnt[q];
       } else if (rec) {
         set_err(w, -ENOSPC);
       }
+      ++idx;
     }
+    __syncthreads();  // warp_tot / base_s reuse
   }
 }
 
@@ -708,7 +816,7 @@ struct Layout {
 
 Layout layout(const gfs_grep_params* p) {
   Layout L{};
-  const uint64_t tcap = pow2_at_least(p->max_words * 2ull < 1024 ? 1024 : p->max_words * 2ull);
+  const uint64_t tcap = pow2_at_least(p->max_words * 8ull < 1024 ? 1024 : p->max_words * 8ull);
   const uint64_t pcap = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap);
   // items: one per chunk of corpus plus one partial chunk per file
   L.max_items = p->corpus_cap / (p->chunk ? p->chunk : 1) + p->max_files + 1;
@@ -737,10 +845,11 @@ Layout layout(const gfs_grep_params* p) {
   return L;
 }
 
-uint32_t scan_smem(uint32_t chunk) {
+uint32_t scan_smem(uint32_t chunk, uint32_t block) {
   const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
   const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
-  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * kCountSlots * 4 + kCountSlots * 2;
+  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * kCountSlots * 4 + kCountSlots * 2 +
+         64 * block;  // token list: <= 32 starts per thread per round (2 bytes each)
 }
 
 }  // namespace
@@ -760,7 +869,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   GrepWork w;
   w.dict = base + L.off[0];
   w.table = (uint64_t*)(base + L.off[1]);
-  w.table_mask = (uint32_t)(pow2_at_least(p->max_words * 2ull < 1024 ? 1024 : p->max_words * 2ull) - 1);
+  w.table_mask = (uint32_t)(pow2_at_least(p->max_words * 8ull < 1024 ? 1024 : p->max_words * 8ull) - 1);
   w.dup_head = (uint32_t*)(base + L.off[2]);
   w.dup_next = (uint32_t*)(base + L.off[3]);
   w.list = base + L.off[4];
@@ -804,7 +913,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   cudaEventRecord(ev, s);
 
   const gfs_ctx* c = gfs_device_ctx(h);
-  const uint32_t smem = scan_smem(p->chunk);
+  const uint32_t smem = scan_smem(p->chunk, p->block);
   if (smem > 227 * 1024) return -EINVAL;
   cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   // GFS_GREP_DEBUG=1: synchronise after each stage, print its time and the first error
@@ -829,6 +938,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   // closed it would re-validate it with the host (close-to-open)
   const uint32_t read_blocks = (uint32_t)(lr < 1024 ? lr : 1024);
   k_grep_init<<<1024, 256, 0, s>>>(w, p->max_words);
+  k_grep_hold<<<1, 32, 0, s>>>(c, d_str, d_str + kMaxPath, w, 0);
   k_grep_dict<<<64, 256, 0, s>>>(c, d_str, w, p->max_words);
   stage("dict");
   k_grep_list_read<<<read_blocks, 256, 0, s>>>(c, d_str + kMaxPath, w, p->list_cap);
@@ -854,7 +964,8 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
       c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
   stage("scan");
   if (!p->keep_open) k_grep_close<<<nsm * 16, 32, 0, s>>>(c, w);
-  k_grep_compact<<<1024, 256, 0, s>>>(w, d_rec, d_rec ? rec_cap : 0, d_totals);
+  k_grep_compact<<<nsm * 8, 256, 0, s>>>(w, d_rec, d_rec ? rec_cap : 0, d_totals);
+  k_grep_hold<<<1, 32, 0, s>>>(c, d_str, d_str + kMaxPath, w, 1);
   k_grep_summary<<<1, 32, 0, s>>>(w, d_summary);
   stage("done");
   const cudaError_t e = cudaGetLastError();

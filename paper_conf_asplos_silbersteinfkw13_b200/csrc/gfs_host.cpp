@@ -36,6 +36,7 @@
 #include <csignal>
 #include <string>
 #include <sys/mman.h>
+#include <sys/prctl.h>
 #include <sys/resource.h>
 #include <sys/stat.h>
 #include <thread>
@@ -201,6 +202,7 @@ struct gfs_handle {
   uint8_t* staging_h = nullptr;
   std::vector<Worker> workers;
   std::atomic<uint64_t> next_ticket{0};
+  std::atomic<uint64_t> frontier{0};  // one past the highest ticket whose request has arrived
   std::atomic<bool> running{false};
   std::mutex fd_mu;  // protects files / free_hfids
   std::vector<HostFile> files;
@@ -567,6 +569,7 @@ void worker_loop(gfs_handle* h, int wi) {
   // A private fd table for this worker (see HostFile): its open()/close()
   // no longer contend with the other workers' on one table lock.
   unshare(CLONE_FILES);
+  prctl(PR_SET_TIMERSLACK, 1000UL);  // idle sleeps end close to when asked (default slack 50 us)
   const uint32_t R = h->h.ring_slots;
   while (h->running.load(std::memory_order_acquire)) {
     const uint64_t t = h->next_ticket.fetch_add(1);
@@ -580,7 +583,10 @@ void worker_loop(gfs_handle* h, int wi) {
         break;
       }
       ++spins;
-      if (spins < 4096) {
+      // The workers holding the next two tickets the GPU will publish poll
+      // without sleeping (one RPC round trip ~ microseconds); the rest back off.
+      const bool hot = t <= h->frontier.load(std::memory_order_relaxed) + 1;
+      if (hot || spins < 4096) {
         cpu_relax();
       } else if (spins < 65536) {
         sched_yield();
@@ -589,6 +595,9 @@ void worker_loop(gfs_handle* h, int wi) {
       }
     }
     if (stop) break;
+    for (uint64_t f = h->frontier.load(std::memory_order_relaxed);
+         f < t + 1 && !h->frontier.compare_exchange_weak(f, t + 1, std::memory_order_relaxed);) {
+    }
     gfs_rpc_req q;
     q.op = vq->op;
     q.hfid = vq->hfid;
@@ -826,6 +835,7 @@ GFS_API int gfs_daemon_stop(gfs_handle* h) {
   cudaMemcpyAsync(&tail, h->h.ring_tail, 8, cudaMemcpyDeviceToHost, h->priv);
   cudaStreamSynchronize(h->priv);
   h->next_ticket.store(tail);
+  h->frontier.store(tail);
   return 0;
 }
 
