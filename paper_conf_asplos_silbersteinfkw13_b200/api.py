@@ -174,32 +174,41 @@ class GpuFS:
         return int(d_ret.item())
 
     # grep -w ------------------------------------------------------------------
+    def grep_state(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
+                   pair_cap=1 << 24, hit_cap=None, corpus_cap=1 << 34, rec_cap=1 << 22):
+        """Device buffers of one grep configuration (allocated once, reused by grep(state=...)).
+        Capacities come from file metadata (stat), never from file contents."""
+        import os
+        torch = _torch()
+        from . import gfs_grep_params, gfs_grep_work_bytes
+        dev = f"cuda:{self.device}"
+        nwords = max(1, os.path.getsize(dict_path) // 32)
+        lbytes = os.path.getsize(list_path)
+        p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
+                            pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 1 << 20, block=block,
+                            keep_open=1 if keep_open else 0, corpus_cap=corpus_cap)
+        if hits:
+            p.hit_cap = hit_cap if hit_cap is not None else 1 << 22
+        work = torch.empty(gfs_grep_work_bytes(p), dtype=torch.uint8, device=dev)
+        rec = torch.empty(3 * rec_cap, dtype=torch.int32, device=dev)
+        totals = torch.empty(nwords, dtype=torch.int64, device=dev)
+        d_hits = torch.empty(2 * max(p.hit_cap, 1), dtype=torch.int64, device=dev) if hits else None
+        summ = torch.zeros(10, dtype=torch.int64, device=dev)
+        return dict(p=p, work=work, rec=rec, rec_cap=rec_cap, totals=totals, hits=d_hits, summary=summ)
+
     def grep(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
              pair_cap=1 << 24, hit_cap=None, stream=None, sync=True, state=None, corpus_cap=1 << 34,
              rec_cap=1 << 22):
         """grep -w. Returns a dict with records (n,3) sorted by (file, word),
         totals, digest (sum, xor, nhits), hits (n,3) sorted by (file, offset, word) if requested.
+        With sync=False, only enqueues and returns the state (read it after synchronising).
 
         Capacities come from file metadata (stat), never from file contents: the
         contents are read on the GPU through gopen/gread."""
-        import os
-        torch = _torch()
-        from . import GREP_SUMMARY, gfs_grep, gfs_grep_params, gfs_grep_work_bytes
-        dev = f"cuda:{self.device}"
+        from . import GREP_SUMMARY, gfs_grep
         if state is None:
-            nwords = max(1, os.path.getsize(dict_path) // 32)
-            lbytes = os.path.getsize(list_path)
-            p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
-                                pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 1 << 20, block=block,
-                                keep_open=1 if keep_open else 0, corpus_cap=corpus_cap)
-            if hits:
-                p.hit_cap = hit_cap if hit_cap is not None else 1 << 22
-            work = torch.empty(gfs_grep_work_bytes(p), dtype=torch.uint8, device=dev)
-            rec = torch.empty(3 * rec_cap, dtype=torch.int32, device=dev)
-            totals = torch.empty(nwords, dtype=torch.int64, device=dev)
-            d_hits = torch.empty(2 * max(p.hit_cap, 1), dtype=torch.int64, device=dev) if hits else None
-            summ = torch.zeros(10, dtype=torch.int64, device=dev)
-            state = dict(p=p, work=work, rec=rec, rec_cap=rec_cap, totals=totals, hits=d_hits, summary=summ)
+            state = self.grep_state(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap, hit_cap,
+                                    corpus_cap, rec_cap)
         p = state["p"]
         s, sp = self._stream(stream)
         gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),

@@ -79,6 +79,7 @@ struct GrepWork {
   uint64_t pair_mask;
   // counters
   unsigned long long* vars;  // see V_*
+  unsigned long long* prof;  // GFS_GREP_PROF=1: per-phase cycles of k_grep_scan thread 0 (else null)
 };
 enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS, V_DSUM, V_DXOR, V_NLISTED,
        V_NEXTF, V_LISTSZ, V_HOLD_DICT, V_HOLD_LIST, V_NVARS };
@@ -110,18 +111,21 @@ __device__ __forceinline__ uint32_t word_bits32(const uint8_t* p) {
          (word_bits4(b.x) << 16) | (word_bits4(b.y) << 20) | (word_bits4(b.z) << 24) | (word_bits4(b.w) << 28);
 }
 
-// Hash of a word given as 8 little-endian 32-bit words, zero-padded past its
-// length L (dictionary slots and tokens are both brought to this form).
-__device__ __forceinline__ uint64_t tok_hash(const uint32_t (&v)[8], uint32_t L) {
-  uint64_t h = 0x9E3779B97F4A7C15ull * (L + 1);
-#pragma unroll
-  for (int j = 0; j < 4; ++j) {
-    h ^= ((uint64_t)v[2 * j + 1] << 32) | v[2 * j];
-    h *= 0xBF58476D1CE4E5B9ull;
-    h ^= h >> 29;
-  }
+// Hash of a word from its first 8 bytes (zero-padded past its length L) and
+// L. Longer words sharing a prefix and length collide on purpose: every key
+// match is confirmed by an exact 32-byte compare, and the table keeps each
+// such word in its own entry (k_grep_dict), so lookups stay exact.
+__device__ __forceinline__ uint64_t tok_hash(uint32_t w0, uint32_t w1, uint32_t L) {
+  uint64_t h = (((uint64_t)w1 << 32) | w0) ^ (0x9E3779B97F4A7C15ull * L);
+  h *= 0xBF58476D1CE4E5B9ull;
+  h ^= h >> 29;
   h *= 0x94D049BB133111EBull;
   return h ^ (h >> 32);
+}
+
+// Low `nb` (0..4) bytes of a word.
+__device__ __forceinline__ uint32_t low_bytes(uint32_t x, int nb) {
+  return x & __funnelshift_lc(0xFFFFFFFFu, 0u, 8 * nb);
 }
 
 // Bytes [0, L) of the 32 starting at byte offset `sh` (0..15) of 12 words,
@@ -155,8 +159,13 @@ __device__ __forceinline__ uint64_t splitmix64(uint64_t x) {
 }
 
 // Order-independent digest term of one hit (file f, byte offset off, word k).
-__device__ __forceinline__ uint64_t hit_mix(uint64_t f, uint64_t off, uint64_t k) {
+// The digest term of one hit (R20); hit_mix_hf below is the form the scan uses.
+__device__ __forceinline__ __attribute__((unused)) uint64_t hit_mix(uint64_t f, uint64_t off, uint64_t k) {
   return splitmix64(splitmix64(splitmix64(f) + off) + k);
+}
+// The same with splitmix64(f) computed once per file (hf).
+__device__ __forceinline__ uint64_t hit_mix_hf(uint64_t hf, uint64_t off, uint64_t k) {
+  return splitmix64(splitmix64(hf + off) + k);
 }
 
 __device__ __forceinline__ void set_err(GrepWork& w, long long e) { atomicMin((long long*)&w.vars[V_ERR], e); }
@@ -219,10 +228,7 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
         // zero the bytes after the word: the slot becomes the word's padded form
         // (other threads only ever read bytes [0, n) of a slot of length n)
         for (uint32_t i = n; i < 32; ++i) s[i] = 0;
-        uint32_t v[8];
-#pragma unroll
-        for (int j = 0; j < 8; ++j) v[j] = ((const uint32_t*)s)[j];
-        const uint64_t h = tok_hash(v, n);
+        const uint64_t h = tok_hash(((const uint32_t*)s)[0], ((const uint32_t*)s)[1], n);
         const uint64_t ent = entry_key(h, n) | (k + 1);
         // linear probing from the start of the hash's 4-entry (32-byte) bucket:
         // lookups read a whole bucket per step (scan_token)
@@ -454,6 +460,7 @@ struct ScanSmem {
   uint32_t* ckey;   // count table: word + 1 (0 = empty)
   uint32_t* ccnt;
   uint16_t* olist;  // occupied count slots, in insertion order
+  uint64_t hf;      // splitmix64(file index) of the current item (digest)
 };
 
 // One hit of word k at file position pos: per-item shared count (spilling to
@@ -476,7 +483,7 @@ __device__ __forceinline__ void count_hit(GrepWork& w, const ScanSmem& S, uint32
     pair_add(w, f, k, 1);
     *spilled = 1;
   }
-  const uint64_t m = hit_mix(f, pos, k);
+  const uint64_t m = hit_mix_hf(S.hf, pos, k);
   acc.dsum += m;
   acc.dxor ^= m;
   ++acc.nh;
@@ -493,19 +500,12 @@ __device__ __forceinline__ void count_hit(GrepWork& w, const ScanSmem& S, uint32
 __device__ __forceinline__ void scan_token(GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
                                            uint32_t f, uint32_t i, uint32_t L, uint64_t pos, uint64_t* hits,
                                            uint64_t hit_cap, ScanAcc& acc) {
-  uint32_t W[12];
-  const uint4* q = (const uint4*)(S.buf + (i & ~15u));
-#pragma unroll
-  for (int j = 0; j < 3; ++j) {
-    const uint4 t = q[j];
-    W[4 * j] = t.x;
-    W[4 * j + 1] = t.y;
-    W[4 * j + 2] = t.z;
-    W[4 * j + 3] = t.w;
-  }
-  uint32_t v[8];
-  gather_token(W, i & 15u, L, v);
-  const uint64_t h = tok_hash(v, L);
+  // first 8 bytes: three aligned words and two funnel shifts
+  const uint32_t* a = (const uint32_t*)(S.buf + (i & ~3u));
+  const uint32_t a0 = a[0], a1 = a[1], a2 = a[2], r8 = (i & 3u) * 8;
+  const uint32_t w0 = low_bytes(__funnelshift_r(a0, a1, r8), min((int)L, 4));
+  const uint32_t w1 = low_bytes(__funnelshift_r(a1, a2, r8), min(max((int)L - 4, 0), 4));
+  const uint64_t h = tok_hash(w0, w1, L);
   const uint64_t want = entry_key(h, L) >> 26;
   // One 32-byte bucket (4 entries) per step; insertion filled the first empty
   // slot in the same order, so an empty slot ends the search.
@@ -523,6 +523,20 @@ __device__ __forceinline__ void scan_token(GrepWork& w, const ScanSmem& S, uint3
         const uint32_t kp = (uint32_t)(ent[q] & ((1u << 26) - 1)) - 1;
         const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
         const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
+        uint32_t v[8];  // the whole token, zero-padded: only gathered on a key match
+        {
+          uint32_t W[12];
+          const uint4* qv = (const uint4*)(S.buf + (i & ~15u));
+#pragma unroll
+          for (int j = 0; j < 3; ++j) {
+            const uint4 t = qv[j];
+            W[4 * j] = t.x;
+            W[4 * j + 1] = t.y;
+            W[4 * j + 2] = t.z;
+            W[4 * j + 3] = t.w;
+          }
+          gather_token(W, i & 15u, L, v);
+        }
         const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
                            (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
         if (same) {
@@ -591,11 +605,21 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
     S.ccnt[i] = 0;
   }
   if (tid == 0) prefetch();
+  long long t_prev = clock64();
+  auto lap = [&](int k) {
+    if (w.prof && tid == 0) {
+      const long long t = clock64();
+      atomicAdd(&w.prof[k], (unsigned long long)(t - t_prev));
+      t_prev = t;
+    }
+  };
   for (;;) {
     __syncthreads();
+    lap(0);  // 0: waiting at the loop-top barrier (end of flush)
     const uint64_t item = nxt_item;
     if (item >= nitems) break;
     const uint32_t f = nxt_f;
+    S.hf = splitmix64(f);
     const int fd = nxt_fd;
     const uint64_t size = nxt_size;
     const uint64_t s = (item - nxt_base) * chunk;
@@ -610,6 +634,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
     // moves the span with TMA (s is a multiple of the chunk, itself of 16)
     const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
     const int64_t r = gread(c, fd, ws, we - ws, S.buf + vlo);  // starts with a barrier
+    lap(1);  // 1: gread
     if (r != (int64_t)(we - ws)) {
       if (tid == 0) {
         set_err(w, r < 0 ? r : -EIO);
@@ -623,6 +648,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
       S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
     if (tid == 0) S.mask[nstripe] = 0;
     __syncthreads();
+    lap(2);  // 2: pass 1
     if (tid == 0) prefetch();  // next item's fields, overlapping pass 2
     // pass 2, by rounds of 2 stripes per thread: the starts of tokens in
     // [s, e) = buf[kPre, kPre + e - s) are compacted into `tok`, then every
@@ -662,6 +688,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
         for (uint32_t x = st[q]; x; x &= x - 1) tok[off++] = (uint16_t)(jb + __ffs(x) - 1);
       }
       __syncthreads();
+      lap(3);  // 3: token list
       for (uint32_t q = tid; q < total; q += nthr) {
         const uint32_t i = tok[q], j = i >> 5, b = i & 31;
         const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | S.mask[j];
@@ -669,13 +696,16 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
         if (L <= 32)                                   // no dictionary word is longer (R12)
           scan_token(w, S, &nocc_s, &spilled_s, f, i, L, s + i - kPre, hits, hit_cap, acc);
       }
+      lap(4);  // 4: own tokens
       __syncthreads();  // tok and warp_tot are reused by the next round
+      lap(5);  // 5: waiting for the block's other tokens
     }
     // flush: a whole-file item with no spill owns its records; otherwise merge
     const uint32_t nocc = nocc_s;
     const bool direct = s == 0 && e == size && !spilled_s && rec;
     if (direct && tid == 0 && nocc) rbase_s = atomicAdd(&w.vars[V_NREC], (unsigned long long)nocc);
     __syncthreads();
+    if (w.prof && tid == 0) atomicAdd(&w.prof[7], 1ull);  // 7: items
     for (uint32_t q = tid; q < nocc; q += nthr) {
       const uint32_t cs = S.olist[q];
       const uint32_t k = S.ckey[cs] - 1, cnt = S.ccnt[cs];
@@ -918,6 +948,13 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   // GFS_GREP_DEBUG=1: synchronise after each stage, print its time and the first error
   const bool dbg = getenv("GFS_GREP_DEBUG") && *getenv("GFS_GREP_DEBUG") == '1';
+  static unsigned long long* d_prof = nullptr;
+  w.prof = nullptr;
+  if (getenv("GFS_GREP_PROF") && *getenv("GFS_GREP_PROF") == '1') {
+    if (!d_prof && cudaMalloc((void**)&d_prof, 8 * sizeof(unsigned long long)) != cudaSuccess) d_prof = nullptr;
+    if (d_prof) cudaMemsetAsync(d_prof, 0, 8 * sizeof(unsigned long long), s);
+    w.prof = d_prof;
+  }
   struct timespec ts_prev;
   clock_gettime(CLOCK_MONOTONIC, &ts_prev);
   auto stage = [&](const char* name) {
@@ -959,6 +996,14 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   // persistent scan grid: every resident block slot once (p->grid caps it)
   int occ = 1;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_scan, (int)p->block, smem);
+  // GFS_GREP_BPS=n: at most n scan blocks per SM, the rest of the SM's
+  // L1/shared-memory array left to L1 (dictionary buckets of frequent words)
+  if (getenv("GFS_GREP_BPS")) {
+    const int cap = atoi(getenv("GFS_GREP_BPS"));
+    if (cap > 0 && cap < occ) occ = cap;
+    const int pct = (int)((occ * (uint64_t)(smem + 1024) * 100 + 228 * 1024 - 1) / (228 * 1024));
+    cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributePreferredSharedMemoryCarveout, pct < 100 ? pct : 100);
+  }
   const uint32_t scan_grid = (uint32_t)(occ > 0 ? occ : 1) * (uint32_t)nsm;
   k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
       c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
@@ -968,6 +1013,16 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   k_grep_hold<<<1, 32, 0, s>>>(c, d_str, d_str + kMaxPath, w, 1);
   k_grep_summary<<<1, 32, 0, s>>>(w, d_summary);
   stage("done");
+  if (w.prof) {
+    unsigned long long pv[8];
+    cudaMemcpyAsync(pv, w.prof, sizeof(pv), cudaMemcpyDeviceToHost, s);
+    cudaStreamSynchronize(s);
+    const double tot = (double)(pv[0] + pv[1] + pv[2] + pv[3] + pv[4] + pv[5]) + 1e-9;
+    fprintf(stderr, "gfs_grep[scan prof, thread 0 cycles]: items=%llu loop-top=%.1f%% gread=%.1f%% pass1=%.1f%% "
+            "toklist=%.1f%% tokens=%.1f%% wait-others=%.1f%% (%.0f cycles/item)\n", pv[7], 100 * pv[0] / tot,
+            100 * pv[1] / tot, 100 * pv[2] / tot, 100 * pv[3] / tot, 100 * pv[4] / tot, 100 * pv[5] / tot,
+            tot / (double)(pv[7] ? pv[7] : 1));
+  }
   const cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) fprintf(stderr, "gfs_grep: launch failed: %s\n", cudaGetErrorString(e));
   return e == cudaSuccess ? 0 : -EIO;

@@ -11,7 +11,7 @@ runs = int(os.environ.get("RUNS", "6"))
 c = gen.c4_corpus(f"/dev/shm/gfs_bench_c4_{nf}_{mib}", seed=4, nfiles=nf, total_bytes=mib << 20, nwords=58000)
 s = torch.cuda.Stream()
 with g.GpuFS(cache_bytes=4 << 30, page_size=64 << 10, daemon_threads=12, max_files=1 << 16) as fs:
-    state = None
+    state = fs.grep_state(c["dict"], c["list"], keep_open=True, rec_cap=1 << 24, chunk=chunk, block=block)
     for it in range(runs):
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         with torch.cuda.stream(s):
