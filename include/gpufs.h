@@ -101,7 +101,13 @@ int gfs_info(gfs_handle* h, uint64_t* out, int n);
  *           (requires d_len[i] <= smem_bytes), copied out to d_dst afterwards
  *   mode 3: like mode 2 with the destination at smem + d_off[i] % 16, i.e.
  *           co-aligned with the file offset (requires d_len[i] + 15 <= smem_bytes)
- * then gclose(). If gopen fails every d_ret[i] of that block gets its error. */
+ * then gclose().
+ *   mode 4: warp-collective calls instead (gopen_warp / gread_warp /
+ *           gclose_warp): warp w of the grid issues calls w, w + nwarps, ...
+ *           into global memory. block: a multiple of 32, at most
+ *           32 * GFS_WARP_API_MAX_WARPS (256).
+ *   mode 5: like mode 4 into the warp's own shared buffer of smem_bytes
+ *           (co-aligned at d_off[i] % 16), copied out afterwards. If gopen fails every d_ret[i] of that block gets its error. */
 int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
                   const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
                   int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes);

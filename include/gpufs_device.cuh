@@ -273,6 +273,34 @@ __device__ __forceinline__ Scratch& scratch() {
   return s;
 }
 
+// Call groups. The paper's design point is a warp-level API; its
+// prototype calls per threadblock. Both share one implementation,
+// parameterised by the group: who takes part, how it synchronises, and where
+// its scratch lives. key() identifies the group within a launch (scratch is
+// shared memory, never cleared, so cached state is keyed by grid and group).
+struct BlockGroup {
+  static __device__ __forceinline__ int tid() { return block_tid(); }
+  static __device__ __forceinline__ int nthr() { return block_nthr(); }
+  static __device__ __forceinline__ void sync() { __syncthreads(); }
+  static __device__ __forceinline__ Scratch& sc() { return scratch(); }
+  static __device__ __forceinline__ uint32_t key() { return block_linear(); }
+};
+
+#ifndef GFS_WARP_API_MAX_WARPS
+#define GFS_WARP_API_MAX_WARPS 8  // warp-API blocks have at most 8 warps (scratch: 8 x ~1.2 KiB)
+#endif
+__device__ __forceinline__ Scratch& warp_scratch(int w) {
+  __shared__ Scratch s[GFS_WARP_API_MAX_WARPS];
+  return s[w];
+}
+struct WarpGroup {  // every lane of the calling warp takes part (full warps only)
+  static __device__ __forceinline__ int tid() { return block_tid() & 31; }
+  static __device__ __forceinline__ int nthr() { return 32; }
+  static __device__ __forceinline__ void sync() { __syncwarp(); }
+  static __device__ __forceinline__ Scratch& sc() { return warp_scratch(block_tid() >> 5); }
+  static __device__ __forceinline__ uint32_t key() { return (block_linear() << 3) | (uint32_t)(block_tid() >> 5); }
+};
+
 // ------------------------------------------------------------------ staging slots
 // Pinned host memory, page_size bytes per slot, device-mapped; a bitmap in HBM
 // hands slots out. A slot is held only across one RPC and the copy around it,
@@ -605,12 +633,13 @@ __device__ __forceinline__ void mbar_wait(uint64_t* m, uint32_t phase) {
 // The block's mbarrier lives in `Scratch` (static shared memory, not cleared
 // between launches): (re)initialise it the first time this block of this launch
 // needs it. Called by thread 0 only, before the barrier that publishes it.
+template <class G = BlockGroup>
 __device__ __forceinline__ void ensure_mbar(Scratch& sc) {
-  if (sc.mbar_grid != grid_id() || sc.mbar_blk != block_linear()) {
+  if (sc.mbar_grid != grid_id() || sc.mbar_blk != G::key()) {
     mbar_init(&sc.mbar);
     sc.mbar_phase = 0;
     sc.mbar_grid = grid_id();
-    sc.mbar_blk = block_linear();
+    sc.mbar_blk = G::key();
   }
 }
 
@@ -980,9 +1009,10 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
 // retried after the block's own fills, so no block waits on another while it
 // holds an unfilled frame. Returns 0 with every sc.frame[i] held, or -errno
 // with none held.
+template <class G = BlockGroup>
 __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, uint64_t pb, uint32_t cnt,
                              bool first_done) {
-  const int tid = block_tid(), nthr = block_nthr();
+  const int tid = G::tid(), nthr = G::nthr();
   const bool fast = !(c->flags & GFS_F_LOCKED_TRAVERSAL);
   if (!first_done && tid < (int)cnt) sc.frame[tid] = kBusy;
   const uint64_t t0 = now_ns();
@@ -1009,7 +1039,7 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
           sc.nbytes[tid] = r.nbytes;
         }
       }
-      __syncthreads();
+      G::sync();
     }
     int err = 0;
     bool busy = false, pull = false;
@@ -1025,7 +1055,7 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
           block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), stage_ptr(c, sc.stage[i]), sc.nbytes[i],
                                       tid, nthr);
       __threadfence();
-      __syncthreads();
+      G::sync();
       if (tid < (int)cnt && sc.frame[tid] >= 0 && sc.fill[tid] && sc.stage[tid] >= 0) {
         const uint32_t f = (uint32_t)sc.frame[tid];
         stage_free(c, sc.stage[tid]);
@@ -1041,11 +1071,11 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
         if (sc.fill[tid]) frame_retire(c, f, GFS_ST_FILLING);  // an installed O_GWRONCE page nobody wrote
         frame_release(c, f);
       }
-      __syncthreads();
+      G::sync();
       return err;
     }
     if (!busy) {
-      if (pull) __syncthreads();
+      if (pull) G::sync();
       return 0;
     }
     // still busy: back off and retry (the timeout decision is made by one
@@ -1053,11 +1083,11 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
     if (tid == 0) sc.busy = timed_out(c, t0) ? 1u : 0u;
     if (tid < 32) __nanosleep(ns);
     ns = ns < 2048 ? ns * 2 : 2048;
-    __syncthreads();
+    G::sync();
     if (sc.busy) {
       if (tid == 0) ctr(c, GFS_C_TIMEOUT);
       if (tid < (int)cnt && sc.frame[tid] == kBusy) sc.frame[tid] = -ETIMEDOUT;  // error path next round
-      __syncthreads();
+      G::sync();
     }
   }
 }
@@ -1128,8 +1158,9 @@ __device__ __forceinline__ bool snap_fd(const gfs_ctx* c, int fd, FileSnap* s) {
 
 // Snapshot for gread: read-only files this block opened are served from the
 // block's cached snapshot (their entry cannot change while held open).
+template <class G = BlockGroup>
 __device__ __forceinline__ bool snap_fd_cached(const gfs_ctx* c, Scratch& sc, int fd, FileSnap* s) {
-  if (sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id()) {
+  if (sc.cached_fd == fd && sc.cached_blk == G::key() && sc.cached_grid == grid_id()) {
     *s = sc.cached;
     return true;
   }
@@ -1438,13 +1469,14 @@ using detail::Scratch;
 // flags: GFS_O_RDONLY or GFS_O_GWRONCE, optionally | GFS_O_PREFETCH (hint:
 // when the open goes to the host, page 0 comes back with the reply and the
 // calling block installs it — one RPC instead of two for small files).
-__device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
-  Scratch& sc = detail::scratch();
-  const int tid = detail::block_tid();
-  __syncthreads();
+template <class G>
+__device__ inline int gopen_t(const gfs_ctx* c, const char* path, int flags) {
+  Scratch& sc = G::sc();
+  const int tid = G::tid();
+  G::sync();
   uint64_t ph = 0;
   uint32_t pn = 0;
-  if (detail::block_nthr() >= 32) {  // warp 0 measures and hashes the path together
+  if (G::nthr() >= 32) {  // warp 0 measures and hashes the path together
     if (tid < 32) pn = detail::path_len_hash_warp(path, &ph);
   } else if (tid == 0) {
     pn = detail::path_len_hash(path, &ph);
@@ -1459,19 +1491,19 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
     sc.cached_fd = -1;
     if (fd >= 0 && detail::snap_fd(c, fd, &sc.cached) && !(sc.cached.oflags & GFS_O_GWRONCE)) {
       sc.cached_grid = detail::grid_id();
-      sc.cached_blk = detail::block_linear();
+      sc.cached_blk = G::key();
       sc.cached_fd = fd;
       for (int i = 0; i < detail::kLeafCache; ++i) sc.leaf[i] = 0;
     }
-    detail::ensure_mbar(sc);
+    detail::ensure_mbar<G>(sc);
   }
-  __syncthreads();
+  G::sync();
   if (sc.frame[0] >= 0) {  // pull the prefetched page 0 and publish it
     const uint32_t f = (uint32_t)sc.frame[0];
     detail::block_copy_from_frame<true>(detail::frame_ptr(c, f), detail::stage_ptr(c, sc.stage[0]), sc.nbytes[0],
-                                        tid, detail::block_nthr());
+                                        tid, G::nthr());
     __threadfence();
-    __syncthreads();
+    G::sync();
     if (tid == 0) {
       detail::stage_free(c, sc.stage[0]);
       detail::st_rlx(&c->f_valid[f], sc.nbytes[0]);
@@ -1479,51 +1511,54 @@ __device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
       detail::frame_release(c, f);
       sc.frame[0] = -1;
     }
-    __syncthreads();
+    G::sync();
   }
   return (int)sc.ret;
 }
 
 // gclose: drops this block's reference; never writes back.
-__device__ inline int gclose(const gfs_ctx* c, int fd) {
-  Scratch& sc = detail::scratch();
-  __syncthreads();
-  if (detail::block_tid() == 0) {
+template <class G>
+__device__ inline int gclose_t(const gfs_ctx* c, int fd) {
+  Scratch& sc = G::sc();
+  G::sync();
+  if (G::tid() == 0) {
     if (sc.cached_fd == fd) sc.cached_fd = -1;
     sc.ret = detail::close_leader(c, fd);
   }
-  __syncthreads();
+  G::sync();
   return (int)sc.ret;
 }
 
-__device__ inline int64_t gfstat_size(const gfs_ctx* c, int fd) {
-  Scratch& sc = detail::scratch();
-  __syncthreads();
-  if (detail::block_tid() == 0) {
+template <class G>
+__device__ inline int64_t gfstat_size_t(const gfs_ctx* c, int fd) {
+  Scratch& sc = G::sc();
+  G::sync();
+  if (G::tid() == 0) {
     detail::FileSnap s;
     sc.ret = detail::snap_fd(c, fd, &s) ? (int64_t)s.size : -EBADF;
   }
-  __syncthreads();
+  G::sync();
   return sc.ret;
 }
 
 // gread: pread semantics; returns min(len, S-off) bytes, 0 at/after EOF.
-__device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+template <class G>
+__device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
   using namespace detail;
-  Scratch& sc = scratch();
-  const int tid = block_tid(), nthr = block_nthr();
+  Scratch& sc = G::sc();
+  const int tid = G::tid(), nthr = G::nthr();
   const uint32_t shift = c->page_shift;
   const uint64_t P = c->page_size;
   const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
   const bool fast = !(c->flags & GFS_F_LOCKED_TRAVERSAL);
-  __syncthreads();  // the call is a barrier: earlier uses of dst by the block are complete
+  G::sync();  // the call is a barrier: earlier uses of dst by the block are complete
   // Warp 0 alone: snapshot + clip, then the first batch's fast-path lookups
   // (one page per lane). Other warps only touch `sc` after the next barrier.
   if (tid < 32) {
     if (tid == 0) {
-      ensure_mbar(sc);
+      ensure_mbar<G>(sc);
       FileSnap s;
-      const bool cached = sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id();
+      const bool cached = sc.cached_fd == fd && sc.cached_blk == G::key() && sc.cached_grid == grid_id();
       if (cached) s = sc.cached;
       if (!(cached || snap_fd(c, fd, &s)) || (s.oflags & GFS_O_GWRONCE)) {
         sc.ret = -EBADF;
@@ -1571,14 +1606,14 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
     }
     if (tid == 0) sc.quick = quick;
   }
-  __syncthreads();
+  G::sync();
   const int64_t n = sc.ret;
   if (n <= 0) return n;
   if (sc.quick) {
     const uint32_t ph = sc.mbar_phase;
     copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + (off & (P - 1)), (uint32_t)n, tid);
     mbar_wait(&sc.mbar, ph);
-    __syncthreads();
+    G::sync();
     if (tid == 0) {
       sc.mbar_phase = ph ^ 1u;
       frame_release(c, (uint32_t)sc.frame[0]);
@@ -1593,7 +1628,7 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
   const bool tma = __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0;
   for (uint64_t pb = p0; pb <= p1; pb += B) {
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
-    const int err = acquire_batch(c, sc, fs, pb, cnt, pb == p0);
+    const int err = acquire_batch<G>(c, sc, fs, pb, cnt, pb == p0);
     if (err) return err;
     const uint64_t bs = pb == p0 ? (off & (P - 1)) : 0;
     const uint64_t be = pb + cnt - 1 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
@@ -1629,7 +1664,7 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
         }
       }
       mbar_wait(&sc.mbar, ph);
-      __syncthreads();
+      G::sync();
       if (tid == 0) sc.mbar_phase = ph ^ 1u;
     } else {
       for (uint32_t i = 0; i < cnt; ++i) {
@@ -1639,11 +1674,37 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
         block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
                               e - s, tid, nthr);
       }
-      __syncthreads();
+      G::sync();
     }
     if (tid < (int)cnt) frame_release(c, (uint32_t)sc.frame[tid]);
   }
   return n;
+}
+
+// Threadblock-collective calls (the prototype's granularity).
+__device__ inline int gopen(const gfs_ctx* c, const char* path, int flags) {
+  return gopen_t<detail::BlockGroup>(c, path, flags);
+}
+__device__ inline int gclose(const gfs_ctx* c, int fd) { return gclose_t<detail::BlockGroup>(c, fd); }
+__device__ inline int64_t gfstat_size(const gfs_ctx* c, int fd) { return gfstat_size_t<detail::BlockGroup>(c, fd); }
+__device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+  return gread_t<detail::BlockGroup>(c, fd, off, len, dst);
+}
+
+// Warp-collective calls (the paper's design point): every lane of
+// one warp calls with identical arguments; warps of a block proceed
+// independently (no block barrier). Blocks using them have full warps and at
+// most GFS_WARP_API_MAX_WARPS warps. Same semantics and errors as the block
+// calls; `dst` may be global or shared memory.
+__device__ inline int gopen_warp(const gfs_ctx* c, const char* path, int flags) {
+  return gopen_t<detail::WarpGroup>(c, path, flags);
+}
+__device__ inline int gclose_warp(const gfs_ctx* c, int fd) { return gclose_t<detail::WarpGroup>(c, fd); }
+__device__ inline int64_t gfstat_size_warp(const gfs_ctx* c, int fd) {
+  return gfstat_size_t<detail::WarpGroup>(c, fd);
+}
+__device__ inline int64_t gread_warp(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+  return gread_t<detail::WarpGroup>(c, fd, off, len, dst);
 }
 
 // gwrite: pwrite semantics on an O_GWRONCE file.

@@ -80,8 +80,9 @@ class GpuFS:
 
     # gread / gmmap parity harness -------------------------------------------
     def gread_calls(self, path, offs, lens, mode=0, grid=None, block=256, smem=0, stream=None):
-        """Issue gread (mode 0), gmmap (1), gread-to-shared (2) or gread-to-shared co-aligned with the
-        offset (3) calls; returns (ret, dst, dstoff)."""
+        """Issue gread (mode 0), gmmap (1), gread-to-shared (2), gread-to-shared co-aligned with the
+        offset (3), warp-collective gread_warp to global (4) or to per-warp shared (5) calls;
+        returns (ret, dst, dstoff)."""
         torch = _torch()
         offs = np.asarray(offs, dtype=np.uint64)
         lens = np.asarray(lens, dtype=np.uint64)
@@ -95,7 +96,7 @@ class GpuFS:
         d_ret = torch.full((max(n, 1),), -999, dtype=torch.int64, device=f"cuda:{self.device}")
         s, sp = self._stream(stream)
         grid = grid or max(1, min(n, 296))
-        if mode >= 2 and smem == 0:
+        if mode in (2, 3, 5) and smem == 0:
             smem = int(lens.max()) if n else 16
             smem = (smem + 15) // 16 * 16
         gfs_run_gread(self.h, sp, path, mode, n, d_off.data_ptr(), d_len.data_ptr(), d_dstoff.data_ptr(),

@@ -129,6 +129,39 @@ __global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint
   if (fd >= 0) gclose(c, fd);
 }
 
+// Warp-collective variant of the parity harness (gopen_warp / gread_warp /
+// gclose_warp): warp w of the grid issues calls w, w + nwarps, ...
+// mode 4: into global memory; mode 5: into the warp's shared buffer
+// (smem_bytes per warp) at off % 16, then copied out.
+__global__ void k_gread_calls_warp(const gfs_ctx* c, const char* path, int mode, uint32_t ncalls,
+                                   const uint64_t* off, const uint64_t* len, const uint64_t* dstoff, uint8_t* dst,
+                                   int64_t* ret, uint32_t smem_bytes) {
+  extern __shared__ __align__(16) uint8_t smem[];
+  const int lane = threadIdx.x & 31, wib = threadIdx.x >> 5;
+  const uint32_t gw = blockIdx.x * (blockDim.x >> 5) + wib, nw = gridDim.x * (blockDim.x >> 5);
+  uint8_t* wbuf = smem + (size_t)wib * smem_bytes;
+  const int fd = gopen_warp(c, path, GFS_O_RDONLY);
+  for (uint32_t i = gw; i < ncalls; i += nw) {
+    int64_t r;
+    if (fd < 0) {
+      r = fd;
+    } else if (mode == 4) {
+      r = gread_warp(c, fd, off[i], len[i], dst + dstoff[i]);
+    } else {
+      const uint32_t sh = (uint32_t)(off[i] & 15);
+      if (len[i] + sh > smem_bytes) {
+        r = -EINVAL;
+      } else {
+        r = gread_warp(c, fd, off[i], len[i], wbuf + sh);
+        for (int64_t k = lane; k < r; k += 32) dst[dstoff[i] + k] = wbuf[sh + k];
+        __syncwarp();
+      }
+    }
+    if (lane == 0) ret[i] = r;
+  }
+  if (fd >= 0) gclose_warp(c, fd);
+}
+
 __global__ void __launch_bounds__(256, 4) k_seqread(const gfs_ctx* c, const char* path, uint64_t file_off, uint64_t total, uint64_t chunk,
                           int use_mmap, uint8_t* scratch, uint64_t* sum, int64_t* err) {
   const int tid = threadIdx.x, nthr = blockDim.x;
@@ -303,10 +336,20 @@ extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s) {
 GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
                           const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
                           int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes) {
-  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || mode > 3) return -EINVAL;
+  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || mode > 5) return -EINVAL;
+  if (mode >= 4 && ((block & 31) || block > 32 * GFS_WARP_API_MAX_WARPS)) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
   const char* dp = stage_path(path, s);
   if (!dp) return -ENAMETOOLONG;
+  if (mode >= 4) {
+    const uint32_t dyn = mode == 5 ? smem_bytes * (block / 32) : 0;
+    if (dyn > 200 * 1024) return -EINVAL;
+    if (dyn > 48 * 1024)
+      cudaFuncSetAttribute(k_gread_calls_warp, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)dyn);
+    k_gread_calls_warp<<<grid, block, dyn, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len, d_dstoff, d_dst,
+                                                d_ret, smem_bytes);
+    return launch_err(cudaGetLastError());
+  }
   if (mode >= 2 && smem_bytes > 48 * 1024)
     cudaFuncSetAttribute(k_gread_calls, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem_bytes);
   k_gread_calls<<<grid, block, mode >= 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,

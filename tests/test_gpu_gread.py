@@ -114,6 +114,32 @@ def test_gread_into_shared_memory_coaligned(g, shmdir, P):
     check_calls(path, size, offs, lens, ret, dst, dstoff)
 
 
+@pytest.mark.parametrize("mode,P,cache_pages,grid", [
+    # frames >= warps x pages one call holds (the deadlock guard), else < file
+    (4, 4096, 4096, 16),    # warp calls, cache larger than the file
+    (4, 4096, 40, 1),       # warp calls, cache < file: misses, evictions, refetches
+    (4, 65536, 40, 1),
+    (5, 4096, 512, 8),      # warp calls into per-warp shared buffers (TMA middle + edges)
+    (5, 65536, 40, 2),
+])
+def test_gread_warp_api(g, shmdir, mode, P, cache_pages, grid):
+    """gopen_warp / gread_warp / gclose_warp (the paper's warp-level design
+    point): 8 independent warps per block, same bytes as pread."""
+    size = 50 * P + 333
+    path = gen.splitmix_file(os.path.join(shmdir, "w.bin"), size, seed=13)
+    offs, lens = gen.random_calls(17, 500, size, 3 * P, page_size=P)
+    if mode == 5:
+        lens = np.minimum(lens, 8192 - 16)
+    lens[:6] = [0, 1, 15, 17, 4095, 33]
+    offs[:6] = [5, size - 1, 3, P - 7, 1, size + 10]
+    with _fs(g, cache_bytes=cache_pages * P, page_size=P) as fs:
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, mode=mode, grid=grid, block=256,
+                                          smem=8192 if mode == 5 else 0)
+        st = fs.stats()
+    check_calls(path, size, offs, lens, ret, dst, dstoff)
+    assert st["timeout"] == 0 and st["enomem"] == 0
+
+
 @pytest.mark.parametrize("locked", [0, 1])
 def test_locked_traversal_same_bytes(g, shmdir, locked):
     P = 4096
