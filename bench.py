@@ -244,6 +244,9 @@ def run_ours(args):
     mv = None
     if not args.no_matvec:
         mv = matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local)
+    c5 = None
+    if not args.no_c5:
+        c5 = c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist)
 
     tmax = torch.tensor([ms], device=dev)
     if ws > 1:
@@ -283,6 +286,8 @@ def run_ours(args):
         line["grep"] = grep
     if mv:
         line["matvec"] = mv
+    if c5:
+        line["c5"] = c5
     if not args.no_cpu:
         line["cpu_baseline"] = cpu_baseline(args, path, size)
     print(json.dumps(line), flush=True)
@@ -470,6 +475,92 @@ def matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local):
     return out
 
 
+def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
+    """C5 (configs[4]): repeated gwrite/gfsync then re-read across kernel launches.
+    Rank r writes f_r (O_GWRONCE, new content every iteration) and gfsyncs it;
+    after a barrier it re-reads f_{(r+1) % N} twice through its own cache: the
+    first pass re-validates (close-to-open) and misses, the second
+    hits. At N = 1 the file read is the rank's own (re-opened read-only: a fresh
+    incarnation). Parity: the host file equals the source bytes and
+    the GPU read-back checksum equals the oracle's checksum of the host file."""
+    import oracle
+    P = 2 << 20
+    size = args.c5_mib << 20
+    root = "/dev/shm/gfs_bench_c5"
+    os.makedirs(root, exist_ok=True)
+    mine, peer = f"{root}/f_{rank}.bin", f"{root}/f_{(rank + 1) % ws}.bin"
+    base = torch.from_numpy(np.random.default_rng(500 + rank).integers(0, 256, size=size, dtype=np.uint8)).to(dev)
+    src = torch.empty_like(base)
+    grid = 296
+    times = {"write": [], "read_miss": [], "read_hit": []}
+    ok_host, ok_read, errs = True, True, []
+    with g.GpuFS(cache_bytes=4 << 30, page_size=P, device=local, daemon_threads=args.daemon_threads,
+                 max_batch=8, timeout_ms=args.timeout_ms, staging_slots=256) as fs:
+        scratch = torch.empty(grid * P, dtype=torch.uint8, device=dev)
+        out = torch.zeros(2, dtype=torch.int64, device=dev)
+        wout = torch.zeros(2, dtype=torch.int64, device=dev)
+        for it in range(args.c5_iters):
+            src.copy_(base)
+            src.add_(it + 1)  # new content every iteration (mod 256), prepared before the timed region
+            torch.cuda.synchronize()
+            e = [torch.cuda.Event(enable_timing=True) for _ in range(4)]
+            with torch.cuda.stream(stream):
+                e[0].record(stream)
+                fs.seqwrite(mine, src, chunk=P, grid=grid, sync_grid=args.c5_sync_grid, stream=stream, sync=False,
+                            out=wout)
+                e[1].record(stream)
+                stream.synchronize()
+            errs.append(int(wout[0].item()))
+            if ws > 1:
+                dist.barrier()  # every writer has gfsync'ed before anyone re-opens
+            with torch.cuda.stream(stream):
+                out.zero_()
+                e[2].record(stream)
+                fs.seqread(peer, size, P, grid=grid, stream=stream, sync=False, scratch=scratch, out=out)
+                e[3].record(stream)
+                stream.synchronize()
+            s1, err1 = int(out[0].item()) & ((1 << 64) - 1), int(out[1].item())
+            e2 = [torch.cuda.Event(enable_timing=True) for _ in range(2)]
+            with torch.cuda.stream(stream):
+                out.zero_()
+                e2[0].record(stream)
+                fs.seqread(peer, size, P, grid=grid, stream=stream, sync=False, scratch=scratch, out=out)
+                e2[1].record(stream)
+                stream.synchronize()
+            s2, err2 = int(out[0].item()) & ((1 << 64) - 1), int(out[1].item())
+            errs += [err1, err2]
+            times["write"].append(e[0].elapsed_time(e[1]))
+            times["read_miss"].append(e[2].elapsed_time(e[3]))
+            times["read_hit"].append(e2[0].elapsed_time(e2[1]))
+            want = oracle.checksum(peer, 0, size)
+            ok_read &= s1 == want and s2 == want
+            if it == args.c5_iters - 1:
+                hb = np.fromfile(mine, dtype=np.uint8)
+                ok_host &= hb.size == size and np.array_equal(hb, src.cpu().numpy())
+            if ws > 1:
+                dist.barrier()  # nobody rewrites its file while a peer still reads it
+        st = fs.stats()
+    res = {}
+    for k, v in times.items():
+        t = torch.tensor([float(np.median(v))], device=dev)
+        if ws > 1:
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        ms = float(t.item())
+        res[k] = {"ms": round(ms, 3), "GBps": round(ws * size / (ms * 1e-3) / 1e9, 3)}
+    res.update({
+        "workload": f"C5: {args.c5_iters} iterations x (gwrite {args.c5_mib} MiB O_GWRONCE + gfsync from "
+                    f"{args.c5_sync_grid} block(s); barrier; re-read the peer's file twice), 2 MiB pages, 4 GiB "
+                    f"cache, {ws} GPU(s)",
+        "err": min(errs) if errs else 0, "parity": {"host_file": bool(ok_host), "reread_checksums": bool(ok_read)},
+        "counters": {k: st[k] for k in ("miss", "hit", "writeback", "invalidate", "reopen_valid", "rpc_write")},
+        "roofline": {"read_miss": {"bound": "h2d", "peak": round(h2d, 3),
+                                   "frac": round(res["read_miss"]["GBps"] / ws / h2d, 4)},
+                     "read_hit": {"bound": "hbm", "peak": hbm, "note": "2 B HBM per byte (frame read + copy out)",
+                                  "frac": round(2 * res["read_hit"]["GBps"] / ws / hbm, 4)}},
+    })
+    return res
+
+
 def cpu_baseline(args, path, size):
     import oracle
     sample = min(size, args.ref_sample_mib << 20)
@@ -501,6 +592,10 @@ def main():
     ap.add_argument("--no-hit", action="store_true")
     ap.add_argument("--no-grep", action="store_true")
     ap.add_argument("--no-matvec", action="store_true")
+    ap.add_argument("--no-c5", action="store_true")
+    ap.add_argument("--c5-mib", type=int, default=512)
+    ap.add_argument("--c5-iters", type=int, default=3)
+    ap.add_argument("--c5-sync-grid", type=int, default=4)
     ap.add_argument("--mv-rows", type=int, default=11200)  # 5.6 GB (Fig. 8's 5600 MB point x2)
     ap.add_argument("--grep-files", type=int, default=30000)
     ap.add_argument("--grep-mib", type=int, default=500)

@@ -143,6 +143,21 @@ int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncall
  * 3 = gopen+gclose only, 4 = pin (gopen without gclose: the file stays open
  * across launches, *d_ret = fd), 5 = unpin (gclose(fd = arg)).
  * flags = open flags. *d_ret = result. */
+/* C5 write side: pin `path` open O_GWRONCE (one
+ * reference held for the duration), then `grid` blocks gwrite() [0, total)
+ * from device buffer d_src in `chunk`-byte calls (block b takes a contiguous
+ * share), then `sync_grid` blocks call gfsync() on it concurrently (dirty pages
+ * are claimed by CAS, so they split the write-back; -EBUSY from a page another
+ * of them holds is expected) followed, when sync_grid > 1, by one strict
+ * single-block gfsync that must find every page clean, then the pin is dropped
+ * (gclose, no write-back). All on `stream`. *d_err: 0 or the most negative
+ * error (caller zeroes it); d_tmp: one device int64 of scratch (pinned fd).
+ * sync_grid * min(32, block) must not exceed the staging slots (each writing
+ * lane holds one while it waits for its RPC). */
+int gfs_run_seqwrite(gfs_handle* h, void* stream, const char* path, uint64_t total, uint64_t chunk,
+                     const uint8_t* d_src, int64_t* d_err, int64_t* d_tmp, uint32_t grid, uint32_t block,
+                     uint32_t sync_grid);
+
 int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int flags, int op, uint64_t arg,
                    int64_t* d_ret);
 

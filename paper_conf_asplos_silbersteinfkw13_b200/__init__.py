@@ -81,6 +81,7 @@ def lib():
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32], I),
             "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
+            "gfs_run_seqwrite": ([P, P, CS, U64, U64, P, P, P, U32, U32, U32], I),
             "gfs_grep_work_bytes": ([ctypes.POINTER(gfs_grep_params)], U64),
             "gfs_grep": ([P, P, CS, CS, ctypes.POINTER(gfs_grep_params), P, P, U64, P, P, P], I),
             "gfs_matvec": ([P, P, CS, CS, CS, U64, U64, P, P, P, U32, U32], I),
@@ -167,6 +168,11 @@ def gfs_run_seqread(h, stream, path, file_off, total, chunk, use_mmap, d_scratch
 def gfs_run_randread(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):
     return _ck(lib().gfs_run_randread(h, stream, _b(path) if path else None, raw, d_raw, chunk, calls_per_block,
                                       d_off, d_sum, d_err, grid, block), "gfs_run_randread")
+
+
+def gfs_run_seqwrite(h, stream, path, total, chunk, d_src, d_err, d_tmp, grid, block, sync_grid):
+    return _ck(lib().gfs_run_seqwrite(h, stream, _b(path), total, chunk, d_src, d_err, d_tmp, grid, block,
+                                      sync_grid), "gfs_run_seqwrite")
 
 
 def gfs_run_gwrite(h, stream, path, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid, block):

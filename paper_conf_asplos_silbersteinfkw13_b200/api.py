@@ -122,6 +122,24 @@ class GpuFS:
         v = out.cpu().numpy()
         return int(v[0].astype(np.uint64)), int(v[1])
 
+    # sequential gwrite + gfsync (C5 write side) --------------------------------
+    def seqwrite(self, path, src, chunk, grid=148, block=256, sync_grid=1, stream=None, sync=True, out=None):
+        """gwrite the device tensor `src` (uint8) to `path` (O_GWRONCE) from `grid`
+        blocks in `chunk`-byte calls, then gfsync it from `sync_grid` blocks."""
+        torch = _torch()
+        from . import gfs_run_seqwrite
+        if out is None:
+            out = torch.zeros(2, dtype=torch.int64, device=f"cuda:{self.device}")  # [err, pinned fd]
+        else:
+            out.zero_()
+        s, sp = self._stream(stream)
+        gfs_run_seqwrite(self.h, sp, path, src.numel(), chunk, src.data_ptr(), out.data_ptr(), out.data_ptr() + 8,
+                         grid, block, sync_grid)
+        if not sync:
+            return out
+        s.synchronize()
+        return int(out[0].item())
+
     # cache-hit reads into shared memory (K4) ---------------------------------
     def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None):
         torch = _torch()

@@ -266,6 +266,50 @@ __global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncal
   if (fd >= 0) gclose(c, fd);
 }
 
+// C5 write side: every block gopen()s the (pinned, O_GWRONCE) file, gwrite()s
+// its contiguous share of [0, total) from `src` in `chunk`-byte calls, gclose()s.
+__global__ void k_seqwrite(const gfs_ctx* c, const char* path, uint64_t total, uint64_t chunk, const uint8_t* src,
+                           int64_t* err) {
+  const int fd = gopen(c, path, GFS_O_GWRONCE);
+  if (fd < 0) {
+    if (threadIdx.x == 0) note_err(err, fd);
+    return;
+  }
+  const uint64_t nchunks = (total + chunk - 1) / chunk;
+  const uint64_t per = (nchunks + gridDim.x - 1) / gridDim.x;
+  const uint64_t c0 = blockIdx.x * per, c1 = c0 + per < nchunks ? c0 + per : nchunks;
+  for (uint64_t k = c0; k < c1; ++k) {
+    const uint64_t o = k * chunk, n = o + chunk <= total ? chunk : total - o;
+    const int64_t r = gwrite(c, fd, o, n, src + o);
+    if (r != (int64_t)n) {
+      if (threadIdx.x == 0) note_err(err, r < 0 ? r : -EIO);
+      break;
+    }
+  }
+  gclose(c, fd);
+}
+
+// gfsync by every block of the grid: blocks claim dirty pages with a CAS, so
+// concurrent callers split the write-back between them (each waits for its own).
+// allow_busy: -EBUSY (a page claimed by a concurrent gfsync of this grid) is
+// not an error here; a strict single-block pass follows and catches the rest.
+__global__ void k_fsync_from_pin(const gfs_ctx* c, const int64_t* pinned_fd, int64_t* err, int allow_busy) {
+  const int64_t fd = *pinned_fd;
+  if (fd < 0) {
+    if (threadIdx.x == 0 && blockIdx.x == 0) note_err(err, fd);
+    return;
+  }
+  const int r = gfsync(c, (int)fd);
+  if (threadIdx.x == 0 && r < 0 && !(allow_busy && r == -EBUSY)) note_err(err, r);
+}
+
+__global__ void k_unpin(const gfs_ctx* c, const int64_t* pinned_fd, int64_t* err) {
+  const int64_t fd = *pinned_fd;
+  if (fd < 0) return;
+  const int r = gclose(c, (int)fd);
+  if (threadIdx.x == 0 && r < 0) note_err(err, r);
+}
+
 __global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, uint64_t arg, int64_t* ret) {
   if (op == 5) {  // unpin: drop a reference taken by op 4
     const int64_t r = gclose(c, (int)arg);
@@ -391,6 +435,25 @@ GFS_API int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32
   const char* dp = stage_path(path, s);
   if (!dp) return -ENAMETOOLONG;
   k_gwrite_calls<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_seqwrite(gfs_handle* h, void* stream, const char* path, uint64_t total, uint64_t chunk,
+                             const uint8_t* d_src, int64_t* d_err, int64_t* d_tmp, uint32_t grid, uint32_t block,
+                             uint32_t sync_grid) {
+  if (!h || !d_src || !d_err || !d_tmp || grid == 0 || block == 0 || block > 1024 || sync_grid == 0 || chunk == 0)
+    return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = stage_path(path, s);
+  if (!dp) return -ENAMETOOLONG;
+  const gfs_ctx* c = gfs_device_ctx(h);
+  // pin: one open held across the launches, so the writers' gclose never
+  // closes the file (a later O_GWRONCE open would start a new incarnation)
+  k_fileop<<<1, 256, 0, s>>>(c, dp, GFS_O_GWRONCE, 4, 0, d_tmp);
+  k_seqwrite<<<grid, block, 0, s>>>(c, dp, total, chunk, d_src, d_err);
+  k_fsync_from_pin<<<sync_grid, block, 0, s>>>(c, d_tmp, d_err, sync_grid > 1);
+  if (sync_grid > 1) k_fsync_from_pin<<<1, block, 0, s>>>(c, d_tmp, d_err, 0);  // every page clean now
+  k_unpin<<<1, 32, 0, s>>>(c, d_tmp, d_err);
   return launch_err(cudaGetLastError());
 }
 

@@ -153,3 +153,28 @@ def test_more_files_than_fd_cache(g, shmdir):
                         assert fs.unpin(fd) == 0
     finally:
         del os.environ["GFS_FD_CAP"]
+
+
+@pytest.mark.parametrize("P,sync_grid", [(65536, 1), (65536, 4), (1 << 21, 2)])
+def test_c5_write_fsync_reread_iterations(g, shmdir, P, sync_grid):
+    """C5 shape on one cache: each iteration gwrites new content from many blocks,
+    gfsyncs (from sync_grid blocks), then re-reads the file twice through the same
+    cache. The re-open read-only starts a fresh incarnation,
+    so every iteration must see its own bytes: host file == source, GPU read-back
+    checksum == oracle checksum of the host file."""
+    torch = pytest.importorskip("torch")
+    path = os.path.join(shmdir, "c5.bin")
+    size = 24 * P + 4096  # ragged last page
+    with g.GpuFS(cache_bytes=64 * P, page_size=P, timeout_ms=60000, daemon_threads=4,
+                 staging_slots=max(64, 32 * sync_grid)) as fs:
+        for it in range(3):
+            data = np.frombuffer(rnd(size, 100 + it), dtype=np.uint8)
+            src = torch.from_numpy(data.copy()).cuda()
+            assert fs.seqwrite(path, src, chunk=P // 2 + 16, grid=16, sync_grid=sync_grid) == 0
+            assert host(path) == data.tobytes()
+            want = oracle.checksum(path, 0, size)
+            for _ in range(2):  # cold (fresh incarnation: misses) then warm (hits)
+                s, err = fs.seqread(path, size, P, grid=8)
+                assert err == 0 and s == want
+        st = fs.stats()
+    assert st["invalidate"] + st["rpc_open"] >= 3 and st["hit"] > 0
