@@ -595,7 +595,7 @@ def main():
     ap.add_argument("--no-c5", action="store_true")
     ap.add_argument("--c5-mib", type=int, default=512)
     ap.add_argument("--c5-iters", type=int, default=3)
-    ap.add_argument("--c5-sync-grid", type=int, default=4)
+    ap.add_argument("--c5-sync-grid", type=int, default=8)
     ap.add_argument("--mv-rows", type=int, default=11200)  # 5.6 GB (Fig. 8's 5600 MB point x2)
     ap.add_argument("--grep-files", type=int, default=30000)
     ap.add_argument("--grep-mib", type=int, default=500)
