@@ -244,6 +244,9 @@ def run_ours(args):
     mv = None
     if not args.no_matvec:
         mv = matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local)
+    fig4 = None
+    if not args.no_fig4:
+        fig4 = fig4_phase(args, torch, g, dev, stream, h2d, paths, size, local)
     c5 = None
     if not args.no_c5:
         c5 = c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist)
@@ -288,6 +291,8 @@ def run_ours(args):
         line["matvec"] = mv
     if c5:
         line["c5"] = c5
+    if fig4:
+        line["fig4_page_sweep"] = fig4
     if not args.no_cpu:
         line["cpu_baseline"] = cpu_baseline(args, path, size)
     print(json.dumps(line), flush=True)
@@ -475,6 +480,43 @@ def matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local):
     return out
 
 
+def fig4_phase(args, torch, g, dev, stream, h2d, paths, size, local):
+    """Fig. 4 analogue: miss-fill GB/s of a sequential gread sweep
+    against page size. Sweeps alternate between the first 4 GiB of the two C2
+    files with a 2 GiB cache, so every page is a miss (no LRU retention)."""
+    total = min(size, 4 << 30)
+    out = []
+    for pk in (64, 256, 1024, 2048, 4096, 16384):
+        P = pk << 10
+        frames = (2 << 30) // P
+        grid = int(min(296, frames // 2))
+        with g.GpuFS(cache_bytes=2 << 30, page_size=P, device=local, daemon_threads=args.daemon_threads,
+                     timeout_ms=args.timeout_ms, max_batch=min(32, max(1, (8 << 20) // P))) as fs:
+            chunk = max(P, 2 << 20)
+            scratch = torch.empty(grid * chunk, dtype=torch.uint8, device=dev)
+            res = torch.zeros(2, dtype=torch.int64, device=dev)
+            ts = []
+            for rep in range(3):
+                res.zero_()
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                with torch.cuda.stream(stream):
+                    e0.record(stream)
+                    fs.seqread(paths[rep % 2], total, chunk, grid=grid, stream=stream, sync=False, scratch=scratch,
+                               out=res)
+                    e1.record(stream)
+                    stream.synchronize()
+                if rep:
+                    ts.append(e0.elapsed_time(e1))
+            err = int(res[1].item())
+            st = fs.stats()
+        ms = float(np.median(ts))
+        gbs = total / (ms * 1e-3) / 1e9
+        out.append({"page_kib": pk, "GBps": round(gbs, 3), "frac_h2d": round(gbs / h2d, 4), "err": err,
+                    "grid": grid, "misses": st["miss"], "hits": st["hit"]})
+    return {"workload": f"sequential gread sweep of {total >> 30} GiB, 2 GiB cache, chunk max(P, 2 MiB)",
+            "points": out}
+
+
 def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
     """C5 (configs[4]): repeated gwrite/gfsync then re-read across kernel launches.
     Rank r writes f_r (O_GWRONCE, new content every iteration) and gfsyncs it;
@@ -593,6 +635,7 @@ def main():
     ap.add_argument("--no-grep", action="store_true")
     ap.add_argument("--no-matvec", action="store_true")
     ap.add_argument("--no-c5", action="store_true")
+    ap.add_argument("--no-fig4", action="store_true")
     ap.add_argument("--c5-mib", type=int, default=512)
     ap.add_argument("--c5-iters", type=int, default=3)
     ap.add_argument("--c5-sync-grid", type=int, default=8)

@@ -305,7 +305,8 @@ struct WarpGroup {  // every lane of the calling warp takes part (full warps onl
 // Pinned host memory, page_size bytes per slot, device-mapped; a bitmap in HBM
 // hands slots out. A slot is held only across one RPC and the copy around it,
 // never while waiting on another block, so allocation always makes progress.
-__device__ int stage_alloc(const gfs_ctx* c) {
+// wait = false: one pass over the bitmap, -EAGAIN when every slot is taken.
+__device__ int stage_alloc(const gfs_ctx* c, bool wait = true) {
   const uint32_t W = c->staging_words;
   uint32_t w = (smid() * 7u + (uint32_t)(now_ns() >> 6)) % W;
   const uint64_t t0 = now_ns();
@@ -326,6 +327,7 @@ __device__ int stage_alloc(const gfs_ctx* c) {
         cur = prev | (1u << bit);
       }
     }
+    if (!wait) return -EAGAIN;
     waited = true;
     backoff(ns);
     if (timed_out(c, t0)) return -ETIMEDOUT;
@@ -948,17 +950,33 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     }
     if (lk) spin_unlock(lockp);
     if (done) break;
-    // miss (or stale slot): install a new frame for `want`. The slot value
-    // carries the frame's generation, so the CAS cannot succeed against a
-    // value that was replaced and restored in between (no ABA).
+    // miss (or stale slot). A fill needs a staging slot: take one BEFORE
+    // installing anything, without waiting. If none is free the page is
+    // reported busy and retried after this block has pulled (and released)
+    // the pages it did install: a lane never waits for a slot while its block
+    // holds others (hold-and-wait across blocks deadlocked at small pages).
+    const uint64_t base = page << c->page_shift;
+    const uint64_t rem = fs.size > base ? fs.size - base : 0;
+    const uint32_t nb = (fs.oflags & GFS_O_GWRONCE) ? 0u : (uint32_t)(rem < c->page_size ? rem : c->page_size);
+    const int st = nb ? stage_alloc(c, false) : -1;
+    if (nb && st < 0) {
+      ctr(c, GFS_C_STAGE_WAIT);
+      out.frame = kBusy;
+      break;
+    }
+    // Install a new frame for `want`. The slot value carries the frame's
+    // generation, so the CAS cannot succeed against a value that was replaced
+    // and restored in between (no ABA).
     uint32_t gen = 0;
     const int g = alloc_frame(c, want, fs.fdx, &gen);
     if (g < 0) {
+      if (st >= 0) stage_free(c, st);
       out.frame = g;
       break;
     }
     const bool won = a64_cas(slot, s, slot_val((uint32_t)g, gen)) == s;
     if (!won) {
+      if (st >= 0) stage_free(c, st);
       frame_abandon(c, (uint32_t)g);
       ++attempt;
       ctr(c, GFS_C_RETRY);
@@ -970,13 +988,9 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
       ctr(c, GFS_C_ZERO_FILL);
       break;
     }
-    // Fetch min(P, S - pP) bytes: the host preads into a staging slot.
-    const uint64_t base = page << c->page_shift;
-    const uint64_t rem = fs.size > base ? fs.size - base : 0;
-    const uint32_t nb = (uint32_t)(rem < c->page_size ? rem : c->page_size);
-    const int st = nb ? stage_alloc(c) : -1;
-    int32_t r = st < 0 && nb ? st : 0;
-    if (nb && st >= 0) r = rpc_call(c, GFS_OP_READ, fs.hfid, base, st, nb, 0, 0, nullptr, 0, nullptr);
+    // Fetch min(P, S - pP) bytes: the host preads into the staging slot.
+    int32_t r = 0;
+    if (nb) r = rpc_call(c, GFS_OP_READ, fs.hfid, base, st, nb, 0, 0, nullptr, 0, nullptr);
     if (r < 0) {
       if (st >= 0) stage_free(c, st);
       a64_or_rel(&c->f_state[g], GFS_ST_ERROR);
@@ -1330,7 +1344,9 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, uint32_t n, uint6
       // below): every state change is an atomic delta, never a plain store.
       sr_shift(e, GFS_FS_CLAIM, GFS_FS_OPENING, 0);
       gfs_rpc_resp rs;
-      const int pst = (want_pf && flags == (int)GFS_O_RDONLY) ? stage_alloc(c) : -1;
+      // page-0 prefetch only if a staging slot is free right now (never wait
+      // while the entry is OPENING: other openers of the file wait on it)
+      const int pst = (want_pf && flags == (int)GFS_O_RDONLY) ? stage_alloc(c, false) : -1;
       int r = open_rpc_fill(c, e, i, (uint32_t)flags, 0, &rs, pst);
       if (r == 0) r = new_incarnation(c, e, (uint32_t)flags, rs);
       if (r < 0) {
@@ -1798,8 +1814,12 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
   if (fs.oflags & GFS_O_GWRONCE) {
     const uint64_t np = (fs.size + c->page_size - 1) >> c->page_shift;
     const uint32_t B = nthr < 32 ? (uint32_t)nthr : 32u;
-    for (uint64_t pb = 0; pb < np; pb += B) {
+    uint32_t ns = 256;
+    const uint64_t t0 = now_ns();
+    for (uint64_t pb = 0; pb < np;) {
       const uint32_t cnt = (uint32_t)((np - pb) < B ? (np - pb) : B);
+      if (tid == 0) sc.busy = 0;
+      __syncthreads();
       if (tid < (int)cnt) {
         const int f = claim_dirty(c, fs, pb + tid);
         sc.frame[tid] = f;
@@ -1808,12 +1828,15 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
         if (f >= 0) {
           sc.lo[tid] = ld_rlx(&c->f_lo[f]);
           sc.hi[tid] = ld_rlx(&c->f_hi[f]);
-          const int st = stage_alloc(c);
+          // no waiting for a staging slot while holding a claimed page (other
+          // blocks may hold the slots and wait for pages): give the claim
+          // back and redo this batch after the others are written
+          const int st = stage_alloc(c, false);
           sc.stage[tid] = st;
           if (st < 0) {
             a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
             sc.frame[tid] = -1;
-            atomicMin(&sc.err, st);
+            sc.busy = 1;
           }
         }
       }
@@ -1844,6 +1867,16 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
         a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
       }
       __syncthreads();
+      if (!sc.busy) {
+        pb += B;
+        ns = 256;
+      } else {  // some page of the batch found no staging slot: back off, redo the batch
+        if (tid == 0 && timed_out(c, t0)) atomicMin(&sc.err, -ETIMEDOUT);
+        __syncthreads();
+        if (sc.err == -ETIMEDOUT) break;
+        __nanosleep(ns);
+        ns = ns < 8192 ? ns * 2 : 8192;
+      }
     }
   }
   __syncthreads();

@@ -213,6 +213,7 @@ struct gfs_handle {
   std::vector<Worker> workers;
   std::atomic<uint64_t> next_ticket{0};
   std::atomic<uint64_t> frontier{0};  // one past the highest ticket whose request has arrived
+  std::atomic<int64_t> last_arrival_ns{0};  // steady-clock time of the latest request
   std::atomic<bool> running{false};
   std::mutex fd_mu;  // protects files / free_hfids
   std::vector<HostFile> files;
@@ -676,6 +677,7 @@ void worker_loop(gfs_handle* h, int wi) {
     volatile gfs_rpc_req* vq = h->ring_h + slot;
     uint64_t spins = 0;
     bool stop = false;
+    bool hot = false;
     while (__atomic_load_n((const uint64_t*)&vq->seq, __ATOMIC_ACQUIRE) != t + 1) {
       if (!h->running.load(std::memory_order_relaxed)) {
         stop = true;
@@ -683,8 +685,15 @@ void worker_loop(gfs_handle* h, int wi) {
       }
       ++spins;
       // The workers holding the next two tickets the GPU will publish poll
-      // without sleeping (one RPC round trip ~ microseconds); the rest back off.
-      const bool hot = t <= h->frontier.load(std::memory_order_relaxed) + 1;
+      // without sleeping while requests keep coming (one RPC round trip ~
+      // microseconds); after 20 ms without one, and for the other workers,
+      // the pause -> yield -> sleep ladder applies.
+      if ((spins & 255) == 1) {
+        const int64_t now = std::chrono::duration_cast<std::chrono::nanoseconds>(
+                                std::chrono::steady_clock::now().time_since_epoch()).count();
+        hot = t <= h->frontier.load(std::memory_order_relaxed) + 1 &&
+              now - h->last_arrival_ns.load(std::memory_order_relaxed) < 20000000;
+      }
       if (hot || spins < 4096) {
         cpu_relax();
       } else if (spins < 65536) {
@@ -697,6 +706,9 @@ void worker_loop(gfs_handle* h, int wi) {
     for (uint64_t f = h->frontier.load(std::memory_order_relaxed);
          f < t + 1 && !h->frontier.compare_exchange_weak(f, t + 1, std::memory_order_relaxed);) {
     }
+    h->last_arrival_ns.store(std::chrono::duration_cast<std::chrono::nanoseconds>(
+                                 std::chrono::steady_clock::now().time_since_epoch()).count(),
+                             std::memory_order_relaxed);
     gfs_rpc_req q;
     q.op = vq->op;
     q.hfid = vq->hfid;

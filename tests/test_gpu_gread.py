@@ -228,3 +228,19 @@ def test_mapped_reads_and_external_shrink(g, shmdir):
         assert ret[0] == 2 * P  # the open file's size is the one seen at gopen
         assert not dst[:2 * P].any()
         fs.unpin(pfd)
+
+
+def test_few_staging_slots_many_missing_pages(g, shmdir):
+    """Regression: 64 blocks each missing 16 pages at once with only 32 staging
+    slots. A lane must not wait for a slot while its block holds others (that
+    hold-and-wait deadlocked until the timeout); it reports the page busy and
+    retries after its block has pulled the pages it did get."""
+    P = 4096
+    size = 64 * 16 * P * 2
+    path = gen.splitmix_file(os.path.join(shmdir, "st.bin"), size, seed=21)
+    with _fs(g, cache_bytes=4096 * P, page_size=P, staging_slots=32, timeout_ms=10000) as fs:
+        for _ in range(2):
+            s, err = fs.seqread(path, size, 16 * P, grid=64)
+            assert err == 0 and s == oracle.checksum(path, 0, size)
+        st = fs.stats()
+    assert st["timeout"] == 0 and st["stage_wait"] > 0
