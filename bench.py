@@ -541,6 +541,16 @@ def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
         scratch = torch.empty(grid * P, dtype=torch.uint8, device=dev)
         out = torch.zeros(2, dtype=torch.int64, device=dev)
         wout = torch.zeros(2, dtype=torch.int64, device=dev)
+        npeers = 0
+        if ws > 1 and not args.no_peers:
+            # NEXT-1: every cache maps the others (CUDA IPC over NVLink); the first
+            # re-read of the neighbour's file is then served from the writer's cache
+            descs = [None] * ws
+            dist.all_gather_object(descs, fs.export())
+            for r, d in enumerate(descs):
+                if r != rank:
+                    fs.attach_peer(d)
+                    npeers += 1
         for it in range(args.c5_iters):
             src.copy_(base)
             src.add_(it + 1)  # new content every iteration (mod 256), prepared before the timed region
@@ -582,6 +592,9 @@ def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
             if ws > 1:
                 dist.barrier()  # nobody rewrites its file while a peer still reads it
         st = fs.stats()
+        local_peer = None
+        if ws == 1 and not args.no_peers:
+            local_peer = c5_local_peer(args, torch, g, fs, mine, size, P, grid, dev, stream, scratch, out)
     res = {}
     for k, v in times.items():
         t = torch.tensor([float(np.median(v))], device=dev)
@@ -594,13 +607,50 @@ def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
                     f"{args.c5_sync_grid} block(s); barrier; re-read the peer's file twice), 2 MiB pages, 4 GiB "
                     f"cache, {ws} GPU(s)",
         "err": min(errs) if errs else 0, "parity": {"host_file": bool(ok_host), "reread_checksums": bool(ok_read)},
-        "counters": {k: st[k] for k in ("miss", "hit", "writeback", "invalidate", "reopen_valid", "rpc_write")},
-        "roofline": {"read_miss": {"bound": "h2d", "peak": round(h2d, 3),
-                                   "frac": round(res["read_miss"]["GBps"] / ws / h2d, 4)},
+        "counters": {k: st[k] for k in ("miss", "hit", "writeback", "invalidate", "reopen_valid", "rpc_write",
+                                        "rpc_read", "peer_fill", "bytes_peer")},
+        "peers_attached": npeers,
+        "roofline": {"read_miss": ({"bound": "h2d", "peak": round(h2d, 3),
+                                    "frac": round(res["read_miss"]["GBps"] / ws / h2d, 4)} if not npeers else
+                                   {"bound": "nvlink", "peak": 900.0, "unit": "GB/s",
+                                    "peak_source": "nominal NVLink 5 per-direction bandwidth per GPU",
+                                    "frac": round(res["read_miss"]["GBps"] / ws / 900.0, 4)}),
                      "read_hit": {"bound": "hbm", "peak": hbm, "note": "2 B HBM per byte (frame read + copy out)",
                                   "frac": round(2 * res["read_hit"]["GBps"] / ws / hbm, 4)}},
     })
+    if local_peer:
+        res["read_peer_same_gpu"] = local_peer
     return res
+
+
+def c5_local_peer(args, torch, g, fs, path, size, P, grid, dev, stream, scratch, out):
+    """N = 1 stand-in for NEXT-1 (peer-cache fill): a second cache on the same GPU
+    attaches `fs` as its peer and reads the file `fs` holds; every page is copied
+    frame-to-frame (HBM -> HBM here; over NVLink between GPUs). Parity: the
+    checksum equals the oracle's over the host file."""
+    import oracle
+    want = oracle.checksum(path, 0, size)
+    times, ok, st = [], True, {}
+    for rep in range(3):
+        with g.GpuFS(cache_bytes=4 << 30, page_size=P, device=fs.device, daemon_threads=2, max_batch=8,
+                     timeout_ms=args.timeout_ms) as B:
+            B.attach_peer(fs.export())
+            torch.cuda.synchronize()
+            e = [torch.cuda.Event(enable_timing=True) for _ in range(2)]
+            with torch.cuda.stream(stream):
+                out.zero_()
+                e[0].record(stream)
+                B.seqread(path, size, P, grid=grid, stream=stream, sync=False, scratch=scratch, out=out)
+                e[1].record(stream)
+                stream.synchronize()
+            ok &= (int(out[0].item()) & ((1 << 64) - 1)) == want and int(out[1].item()) == 0
+            times.append(e[0].elapsed_time(e[1]))
+            st = B.stats()
+    ms = float(np.median(times))
+    return {"ms": round(ms, 3), "GBps": round(size / (ms * 1e-3) / 1e9, 3), "parity": bool(ok),
+            "peer_fill": st["peer_fill"], "bytes_peer": st["bytes_peer"], "rpc_read": st["rpc_read"],
+            "note": "second cache on the same GPU attached as a peer (NEXT-1 protocol; the copy is HBM->HBM, "
+                    "not NVLink); includes the reader's gopen (OPEN RPC)"}
 
 
 def cpu_baseline(args, path, size):
@@ -644,6 +694,7 @@ def main():
     ap.add_argument("--grep-mib", type=int, default=500)
     ap.add_argument("--grep-cache-gib", type=int, default=4)
     ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--no-peers", action="store_true", help="C5 without peer-cache fill (NEXT-1)")
     args = ap.parse_args()
     if args.impl == "reference":
         run_reference(args)

@@ -74,6 +74,36 @@ int gfs_shutdown(gfs_handle* h);
 /* Device pointer to the gfs_ctx to pass to kernels using gpufs_device.cuh. */
 const gfs_ctx* gfs_device_ctx(gfs_handle* h);
 
+/* ---- peer caches (NEXT-1; the cache "spans multiple GPUs", P:L136-137,
+ * P:L452-454). Each GPU keeps its own cache (one process per GPU);
+ * a cache that attaches its peers fills an O_RDONLY miss from a peer frame
+ * over NVLink when the peer holds the same host file at the same
+ * close-to-open version, clean and host-verified, and asks
+ * the host otherwise. Results are identical either way. */
+typedef struct gfs_export_desc {
+  uint64_t magic;
+  int32_t pid, device;
+  uint32_t page_shift, nframes, max_nodes, max_files;
+  uint64_t ptr[7];              /* exporter's device pointers (same-process attach) */
+  unsigned char ipc[7][64];     /* cudaIpcMemHandle_t of: pool, f_state, f_tag, f_lo, f_hv, nodes, files */
+} gfs_export_desc;
+
+/* Describe this cache for gfs_attach_peer in another process (or handle) and
+ * switch its fills to system-scope publication. Plain bytes: send them to
+ * the peer with any transport (e.g. torch.distributed all_gather_object).
+ * Call before any kernel uses the context. -ENOTSUP if the frame pool is
+ * caller-owned (gfs_config.frame_pool), -EIO if CUDA IPC is unavailable. */
+int gfs_export(gfs_handle* h, gfs_export_desc* out);
+
+/* Map the cache described by `d` (CUDA IPC across processes, direct pointers
+ * within one process, peer access enabled across devices) as a read-only
+ * peer of h. Returns the peer index (>= 0). Same page size required
+ * (-EINVAL); at most GFS_MAX_PEERS (-ENOSPC); -EIO if the mapping fails.
+ * No kernel may use h's context during the call. The exporter must outlive
+ * every kernel of h that runs after the attach (shut h down first, or
+ * barrier). */
+int gfs_attach_peer(gfs_handle* h, const gfs_export_desc* d);
+
 /* Copy the device counters (GFS_C_*, summed over shards) into out[0..n). */
 int gfs_stats(gfs_handle* h, uint64_t* out, int n, int reset);
 

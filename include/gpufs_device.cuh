@@ -188,6 +188,25 @@ __device__ __forceinline__ uint64_t a64_cas(uint64_t* p, uint64_t cmp, uint64_t 
                : "=l"(r) : "l"(p), "l"(cmp), "l"(val) : "memory");
   return r;
 }
+// System-scope variants for another GPU's cache (peer fill): the peer's frame
+// state words are updated by that GPU's threads; NVLink atomics resolve at
+// the owner's L2, and acquire/release must cover both GPUs (.sys).
+__device__ __forceinline__ uint64_t ld_rlx_sys64(const uint64_t* p) {
+  uint64_t v;
+  asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint32_t ld_rlx_sys(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.relaxed.sys.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint64_t a64_add_sys(uint64_t* p, uint64_t v) {
+  uint64_t r;
+  asm volatile("atom.relaxed.sys.global.add.u64 %0, [%1], %2;" : "=l"(r) : "l"(p), "l"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ void fence_sys() { asm volatile("fence.acq_rel.sys;" ::: "memory"); }
 constexpr uint64_t kRefDec = ~0ull;  // ref - 1 (never borrows: the ref being dropped is >= 1)
 __device__ __forceinline__ uint64_t fl64(uint32_t flags) { return ~(uint64_t)flags; }  // and-mask clearing flags
 // Leaf slot value for frame f of generation gen.
@@ -686,12 +705,24 @@ __device__ __forceinline__ uint32_t frame_init(const gfs_ctx* c, uint32_t f, uin
   st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
   st_rlx(&c->f_hi[f], 0);
   st_rlx(&c->f_written[f], 0);
+  st_rlx(&c->f_hv[f], 0);
   st_rlx(&c->f_stamp[f], stamp_now());
   // EVICTING -> FILLING|1 and generation + 1 as one atomic delta: readers that
   // found the frame through a stale slot may hold transient +1s they are about
   // to undo, so the state word is never overwritten with a plain store.
   const uint64_t delta = (1ull << 32) + (uint64_t)GFS_ST_FILLING + 1ull - (uint64_t)GFS_ST_EVICTING;
   return (uint32_t)((a64_add_rel(&c->f_state[f], delta) + delta) >> 32);
+}
+
+// After a successful write-back of [lo, hi) (wr bytes written) that left the
+// host file at `version`: a frame written from byte 0 without holes now equals
+// the host file on [0, hi) (host-verified prefix, peer fill), and the file's
+// synced version advances.
+__device__ __forceinline__ void synced(const gfs_ctx* c, uint32_t f, uint32_t lo, uint32_t hi, uint32_t wr,
+                                       uint64_t version) {
+  st_rlx(&c->f_hv[f], (lo == 0 && wr >= hi) ? hi : 0u);
+  const uint32_t fi = ld_rlx(&c->f_file[f]);
+  if (fi < c->max_files) atomicMax((unsigned long long*)&c->files[fi].synced_version, (unsigned long long)version);
 }
 
 // Write back a frame's dirty range from one thread (the caller owns the frame:
@@ -707,10 +738,12 @@ __device__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t h
   // frame bytes via L2 (.cg): this SM's L1 may hold lines of a previous tenant
   block_copy_from_frame(stage_ptr(c, st) + lo, frame_ptr(c, f) + lo, hi - lo, 0, 1);
   __threadfence_system();
+  gfs_rpc_resp rs;
   const int32_t r = rpc_call(c, GFS_OP_WRITE, hfid, (page << c->page_shift) + lo, st, hi - lo,
-                             wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, nullptr);
+                             wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, &rs);
   stage_free(c, st);
   if (r < 0) return r;
+  synced(c, f, lo, hi, wr, rs.version);
   st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
   st_rlx(&c->f_hi[f], 0);
   st_rlx(&c->f_written[f], 0);
@@ -879,6 +912,87 @@ __device__ __forceinline__ bool peek_busy(const gfs_ctx* c, const FileSnap& fs, 
   return (st >> 32) == (s >> 32) && ((uint32_t)st & (GFS_ST_FILLING | GFS_ST_EVICTING));
 }
 
+// ------------------------------------------------------------------ peer fill
+// NEXT-1 (the buffer cache spans GPUs). On a miss of
+// an O_RDONLY file, before asking the host, look the page up in the peer
+// caches (gfs_peer views of other GPUs' caches, mapped over NVLink). A peer
+// frame is usable iff it holds the same host file (st_ino, st_dev) at the
+// same close-to-open version as this cache's entry, is clean, and its first
+// nb bytes are host-verified (f_hv: filled from the host, or written from
+// byte 0 without holes and then written back). For a peer's O_GWRONCE entry
+// the version is the one its last write-back left (synced_version). Taking
+// the peer frame is the hit protocol of lookup_fast run at system scope: one
+// atomic increment takes the reference and validates the slot's generation;
+// the peer's eviction skips referenced frames. Result code (k << 27) | f, or
+// -1 when no peer has a usable copy.
+constexpr uint32_t kPeerFrameBits = 27;
+__device__ int peer_take(const gfs_ctx* c, const FileSnap& fs, uint64_t page, uint32_t nb) {
+  const gfs_file* me = c->files + fs.fdx;
+  const uint64_t h = ld_rlx64(&me->path_hash);
+  const uint32_t n = ld_rlx(&me->path_len);
+  const uint64_t ino = ld_rlx64(&me->ino), dev = ld_rlx64(&me->dev), ver = ld_rlx64(&me->version);
+  const int64_t mt = (int64_t)ld_rlx64((const uint64_t*)&me->mtime_ns);
+  const uint32_t np = c->npeers;
+  for (uint32_t j = 0; j < np; ++j) {
+    const uint32_t k = (j + (uint32_t)page) % np;  // spread a sweep's pages over the peers
+    const gfs_peer& P = c->peers[k];
+    const uint32_t mask = P.max_files - 1u;
+    uint32_t i = (uint32_t)h & mask;
+    for (uint32_t probe = 0; probe < 64; ++probe, i = (i + 1u) & mask) {
+      gfs_file* e = P.files + i;
+      const uint32_t st = ld_rlx_sys(&e->sr) >> 24;
+      if (st == GFS_FS_FREE) break;
+      if (st != GFS_FS_OPEN && st != GFS_FS_CLOSED) continue;
+      if (ld_rlx_sys64(&e->path_hash) != h || ld_rlx_sys(&e->path_len) != n) continue;
+      if (ld_rlx_sys64(&e->ino) != ino || ld_rlx_sys64(&e->dev) != dev) continue;
+      const uint32_t uid = ld_rlx_sys(&e->uid);
+      const bool wonce = (ld_rlx_sys(&e->oflags) & GFS_O_GWRONCE) != 0;
+      const uint64_t ev = wonce ? ld_rlx_sys64(&e->synced_version) : ld_rlx_sys64(&e->version);
+      if ((wonce && ev == 0) || ev != ver) break;  // the peer's copy is of another version
+      if (!wonce && (ld_rlx_sys64(&e->size) != fs.size || (int64_t)ld_rlx_sys64((const uint64_t*)&e->mtime_ns) != mt))
+        break;
+      const uint32_t height = ld_rlx_sys(&e->height);
+      if (height == 0 || height > GFS_MAX_HEIGHT || (height < 4 && (page >> (GFS_FANOUT_SHIFT * height)) != 0)) break;
+      uint32_t node = ld_rlx_sys(&e->root);
+      for (int lvl = (int)height - 1; lvl >= 1 && node && node < P.max_nodes; --lvl)
+        node = (uint32_t)ld_rlx_sys64(P.nodes + (size_t)node * GFS_FANOUT +
+                                      ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
+      if (!node || node >= P.max_nodes) break;  // type-stable nodes: a racing free reads as a miss
+      const uint64_t sl = ld_rlx_sys64(P.nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
+      const uint32_t f = (uint32_t)sl - 1u;
+      if (!(uint32_t)sl || f >= P.nframes) break;
+      const uint64_t old = a64_add_sys(&P.f_state[f], 1ull);
+      fence_sys();  // the checks and the copy below read after the reference is held
+      if ((old >> 32) == (sl >> 32) && !((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR)) &&
+          ld_rlx_sys64(&P.f_tag[f]) == (((uint64_t)uid << 32) | (uint32_t)page) &&
+          ld_rlx_sys(&P.f_lo[f]) == GFS_DIRTY_NONE && ld_rlx_sys(&P.f_hv[f]) >= nb)
+        return (int)((k << kPeerFrameBits) | f);
+      a64_add_sys(&P.f_state[f], kRefDec);
+      break;
+    }
+  }
+  ctr(c, GFS_C_PEER_MISS);
+  return -1;
+}
+__device__ __forceinline__ const uint8_t* peer_frame_ptr(const gfs_ctx* c, int code) {
+  const gfs_peer& P = c->peers[(uint32_t)code >> kPeerFrameBits];
+  return P.pool + ((size_t)((uint32_t)code & ((1u << kPeerFrameBits) - 1u)) << P.page_shift);
+}
+__device__ __forceinline__ void peer_release(const gfs_ctx* c, int code) {
+  const gfs_peer& P = c->peers[(uint32_t)code >> kPeerFrameBits];
+  a64_add_sys(&P.f_state[(uint32_t)code & ((1u << kPeerFrameBits) - 1u)], kRefDec);
+}
+// Lk.stage / Scratch.stage: >= 0 staging slot, -1 nothing to pull, <= -2 peer frame
+__device__ __forceinline__ int peer_stage(int code) { return -2 - code; }
+__device__ __forceinline__ int stage_peer(int stage) { return -2 - stage; }
+__device__ __forceinline__ const uint8_t* fill_src(const gfs_ctx* c, int stage) {
+  return stage >= 0 ? stage_ptr(c, stage) : peer_frame_ptr(c, stage_peer(stage));
+}
+__device__ __forceinline__ void fill_src_free(const gfs_ctx* c, int stage) {
+  if (stage >= 0) stage_free(c, stage);
+  else peer_release(c, stage_peer(stage));
+}
+
 struct Lk {
   int frame;   // >= 0 held (ref taken); kBusy; or -errno
   int stage;   // >= 0: pull nbytes from this staging slot into the frame
@@ -958,8 +1072,17 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     const uint64_t base = page << c->page_shift;
     const uint64_t rem = fs.size > base ? fs.size - base : 0;
     const uint32_t nb = (fs.oflags & GFS_O_GWRONCE) ? 0u : (uint32_t)(rem < c->page_size ? rem : c->page_size);
-    const int st = nb ? stage_alloc(c, false) : -1;
-    if (nb && st < 0) {
+    // A peer GPU's cache may hold the page (NEXT-1): then no staging slot
+    // and no RPC; `st` names the peer frame (held) instead.
+    const int pc = (nb && c->npeers) ? peer_take(c, fs, page, nb) : -1;
+    int st = -1;
+    if (pc >= 0) {
+      st = peer_stage(pc);
+    } else if (nb) {
+      st = stage_alloc(c, false);
+      if (st < 0) st = -1;  // -EAGAIN: every slot taken
+    }
+    if (nb && st == -1) {
       ctr(c, GFS_C_STAGE_WAIT);
       out.frame = kBusy;
       break;
@@ -970,13 +1093,13 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     uint32_t gen = 0;
     const int g = alloc_frame(c, want, fs.fdx, &gen);
     if (g < 0) {
-      if (st >= 0) stage_free(c, st);
+      if (st != -1) fill_src_free(c, st);
       out.frame = g;
       break;
     }
     const bool won = a64_cas(slot, s, slot_val((uint32_t)g, gen)) == s;
     if (!won) {
-      if (st >= 0) stage_free(c, st);
+      if (st != -1) fill_src_free(c, st);
       frame_abandon(c, (uint32_t)g);
       ++attempt;
       ctr(c, GFS_C_RETRY);
@@ -986,6 +1109,13 @@ __device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
     out.fill = 1;
     if (fs.oflags & GFS_O_GWRONCE) {
       ctr(c, GFS_C_ZERO_FILL);
+      break;
+    }
+    if (pc >= 0) {  // the block copies the peer frame over NVLink
+      out.stage = st;
+      out.nbytes = nb;
+      ctr(c, GFS_C_PEER_FILL);
+      ctr(c, GFS_C_BYTES_PEER, nb);
       break;
     }
     // Fetch min(P, S - pP) bytes: the host preads into the staging slot.
@@ -1061,21 +1191,23 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
       const int f = sc.frame[i];
       if (f == kBusy) busy = true;
       else if (f < 0) err = f;
-      else if (sc.fill[i] && sc.stage[i] >= 0) pull = true;
+      else if (sc.fill[i] && sc.stage[i] != -1) pull = true;
     }
-    if (pull) {  // fill the frames this block installed: staging -> frame over PCIe
+    if (pull) {  // fill the frames this block installed: staging -> frame over PCIe, or peer frame -> frame
       for (uint32_t i = 0; i < cnt; ++i)
-        if (sc.frame[i] >= 0 && sc.fill[i] && sc.stage[i] >= 0)
-          block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), stage_ptr(c, sc.stage[i]), sc.nbytes[i],
+        if (sc.frame[i] >= 0 && sc.fill[i] && sc.stage[i] != -1)
+          block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), fill_src(c, sc.stage[i]), sc.nbytes[i],
                                       tid, nthr);
-      __threadfence();
+      if (c->flags & GFS_F_EXPORTED) __threadfence_system();  // peers read our frames at system scope
+      else __threadfence();
       G::sync();
-      if (tid < (int)cnt && sc.frame[tid] >= 0 && sc.fill[tid] && sc.stage[tid] >= 0) {
+      if (tid < (int)cnt && sc.frame[tid] >= 0 && sc.fill[tid] && sc.stage[tid] != -1) {
         const uint32_t f = (uint32_t)sc.frame[tid];
-        stage_free(c, sc.stage[tid]);
+        fill_src_free(c, sc.stage[tid]);
         sc.stage[tid] = -1;
         sc.fill[tid] = 0;
         st_rlx(&c->f_valid[f], sc.nbytes[tid]);
+        st_rlx(&c->f_hv[f], sc.nbytes[tid]);
         a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));  // publish the page
       }
     }
@@ -1238,6 +1370,7 @@ __device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uin
       st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
       st_rlx(&c->f_hi[f], 0);
       st_rlx(&c->f_written[f], 0);
+      st_rlx(&c->f_hv[f], 0);
       frame_retire(c, f, GFS_ST_EVICTING);  // slots naming this generation go stale
     } else {
       a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
@@ -1293,6 +1426,7 @@ __device__ int new_incarnation(const gfs_ctx* c, gfs_file* e, uint32_t flags, co
   e->dev = rs.dev;
   e->mtime_ns = rs.mtime_ns;
   e->oflags = flags;
+  e->synced_version = 0;
   return 0;
 }
 
@@ -1518,11 +1652,13 @@ __device__ inline int gopen_t(const gfs_ctx* c, const char* path, int flags) {
     const uint32_t f = (uint32_t)sc.frame[0];
     detail::block_copy_from_frame<true>(detail::frame_ptr(c, f), detail::stage_ptr(c, sc.stage[0]), sc.nbytes[0],
                                         tid, G::nthr());
-    __threadfence();
+    if (c->flags & GFS_F_EXPORTED) __threadfence_system();
+    else __threadfence();
     G::sync();
     if (tid == 0) {
       detail::stage_free(c, sc.stage[0]);
       detail::st_rlx(&c->f_valid[f], sc.nbytes[0]);
+      detail::st_rlx(&c->f_hv[f], sc.nbytes[0]);
       detail::a64_and_rel(&c->f_state[f], detail::fl64(GFS_ST_FILLING));
       detail::frame_release(c, f);
       sc.frame[0] = -1;
@@ -1851,12 +1987,14 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
         const uint32_t f = (uint32_t)sc.frame[tid];
         const uint32_t lo = sc.lo[tid], hi = sc.hi[tid];
         const uint32_t wr = ld_rlx(&c->f_written[f]);
+        gfs_rpc_resp rs;
         const int32_t r = rpc_call(c, GFS_OP_WRITE, fs.hfid, ((pb + tid) << c->page_shift) + lo, sc.stage[tid],
-                                   hi - lo, wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, nullptr);
+                                   hi - lo, wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, &rs);
         stage_free(c, sc.stage[tid]);
         if (r < 0) {
           atomicMin(&sc.err, r);
         } else {
+          synced(c, f, lo, hi, wr, rs.version);
           st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
           st_rlx(&c->f_hi[f], 0);
           st_rlx(&c->f_written[f], 0);

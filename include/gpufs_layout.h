@@ -34,6 +34,7 @@ extern "C" {
 /* ---- config flags ------------------------------------------------------ */
 #define GFS_F_LOCKED_TRAVERSAL 1u /* K5 ablation: every lookup takes the file lock */
 #define GFS_F_NO_DMA_COMPLETION 2u /* fallback: completion via memcpy instead of stream write-value */
+#define GFS_F_EXPORTED 4u          /* set by gfs_export: frames are published at system scope for peers */
 
 /* ---- frame state word (pframe "state", 64 bits) -------------------------
  * bits 32..63 generation: +1 each time the frame is (re)assigned to a page.
@@ -77,6 +78,8 @@ typedef struct gfs_file {
   uint32_t lock;      /* file spinlock for locked traversal */
   int32_t err;
   uint32_t pad;
+  uint64_t synced_version; /* O_GWRONCE: host version after this cache's last write-back
+                              (peer fill); 0 = none */
 } gfs_file;
 
 /* ---- RPC (§4.3) -------------------------------------------- */
@@ -146,8 +149,28 @@ enum {
   GFS_C_RING_WAIT,      /* ring slot was busy on post */
   GFS_C_BUSY,           /* lookups that found the page being filled/evicted by another block */
   GFS_C_STAGE_WAIT,     /* staging slot allocation had to wait */
+  GFS_C_PEER_FILL,      /* misses filled from a peer GPU's cache (NVLink) instead of the host */
+  GFS_C_BYTES_PEER,     /* bytes copied from peer caches */
+  GFS_C_PEER_MISS,      /* misses for which no peer held a usable copy */
   GFS_C_NCOUNTERS
 };
+
+/* ---- peer caches (NEXT-1: the buffer cache spans GPUs)
+ * A read-only view of another GPU's cache, every pointer valid in THIS
+ * process's address space (CUDA IPC mapping, or the exporter's own pointers
+ * when both caches live in one process). A miss may be filled from a peer
+ * frame over NVLink instead of the host; see gpufs_device.cuh peer_take. */
+#define GFS_MAX_PEERS 8u
+typedef struct gfs_peer {
+  uint8_t* pool;
+  uint64_t* f_state;
+  uint64_t* f_tag;
+  uint32_t* f_lo;
+  uint32_t* f_hv;
+  uint64_t* nodes;
+  gfs_file* files;
+  uint32_t nframes, max_nodes, max_files, page_shift;
+} gfs_peer;
 
 /* ---- the device context (lives in HBM; kernels receive a pointer) ------ */
 typedef struct gfs_ctx {
@@ -164,6 +187,7 @@ typedef struct gfs_ctx {
   uint32_t* f_hi;
   uint32_t* f_written;
   uint32_t* f_stamp;
+  uint32_t* f_hv;     /* bytes [0, hv) equal the host file at the entry's version (peer fill) */
   uint32_t* fresh_next;
   uint32_t* hand;
   /* radix node pool: 64-bit entries (interior: child node id; leaf: gen << 32 | frame + 1) */
@@ -197,6 +221,10 @@ typedef struct gfs_ctx {
   uint32_t max_batch;
   uint64_t timeout_ns;
   unsigned long long* ctr;
+  /* peer caches (device array of npeers views) */
+  const gfs_peer* peers;
+  uint32_t npeers;
+  uint32_t pad_peers;
 } gfs_ctx;
 
 #ifdef __cplusplus

@@ -18,7 +18,7 @@ LIB_PATH = os.path.join(_PKG, "libgpufs.so")
 COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", "writeback", "rpc",
             "rpc_open", "rpc_read", "rpc_write", "bytes_h2d", "bytes_d2h", "open_fast", "reopen_valid",
             "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
-            "ring_wait", "busy", "stage_wait"]
+            "ring_wait", "busy", "stage_wait", "peer_fill", "bytes_peer", "peer_miss"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
                  "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns",
                  "mapped_reads"]
@@ -50,6 +50,13 @@ class gfs_grep_params(ctypes.Structure):
                 ("corpus_cap", ctypes.c_uint64)]
 
 
+class gfs_export_desc(ctypes.Structure):
+    """include/gpufs.h gfs_export_desc: plain bytes describing a cache for gfs_attach_peer."""
+    _fields_ = [("magic", ctypes.c_uint64), ("pid", ctypes.c_int32), ("device", ctypes.c_int32),
+                ("page_shift", ctypes.c_uint32), ("nframes", ctypes.c_uint32), ("max_nodes", ctypes.c_uint32),
+                ("max_files", ctypes.c_uint32), ("ptr", ctypes.c_uint64 * 7), ("ipc", (ctypes.c_ubyte * 64) * 7)]
+
+
 GREP_SUMMARY = ["nrecords", "nhits", "digest_sum", "digest_xor", "nfiles", "nwords", "bytes", "err",
                 "nhits_listed", "nitems"]
 
@@ -76,6 +83,8 @@ def lib():
             "gfs_stats": ([P, P, I, I], I),
             "gfs_host_stats": ([P, P, I], I),
             "gfs_info": ([P, P, I], I),
+            "gfs_export": ([P, ctypes.POINTER(gfs_export_desc)], I),
+            "gfs_attach_peer": ([P, ctypes.POINTER(gfs_export_desc)], I),
             "gfs_run_gread": ([P, P, CS, I, U32, P, P, P, P, P, U32, U32, U32], I),
             "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
@@ -152,6 +161,19 @@ def gfs_info(h: int) -> dict:
     _ck(lib().gfs_info(h, a, 9), "gfs_info")
     return dict(zip(["page_size", "nframes", "max_files", "max_nodes", "ring_slots", "daemon_threads",
                      "staging_slots", "host_next_ticket", "device_ring_tail"], (int(x) for x in a)))
+
+
+def gfs_export(h: int) -> bytes:
+    """Describe cache h for gfs_attach_peer (in this or another process)."""
+    d = gfs_export_desc()
+    _ck(lib().gfs_export(h, ctypes.byref(d)), "gfs_export")
+    return bytes(d)
+
+
+def gfs_attach_peer(h: int, desc: bytes) -> int:
+    """Attach the cache described by `desc` (gfs_export) as a peer of h; returns its index."""
+    d = gfs_export_desc.from_buffer_copy(desc)
+    return _ck(lib().gfs_attach_peer(h, ctypes.byref(d)), "gfs_attach_peer")
 
 
 # ------------------------------------------------------------------ launchers

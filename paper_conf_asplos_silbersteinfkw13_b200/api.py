@@ -8,7 +8,7 @@ from __future__ import annotations
 
 import numpy as np
 
-from . import (DAEMON_SPAWN, gfs_config_default, gfs_daemon, gfs_daemon_stop, gfs_host_stats, gfs_info,
+from . import (DAEMON_SPAWN, gfs_attach_peer, gfs_export, gfs_config_default, gfs_daemon, gfs_daemon_stop, gfs_host_stats, gfs_info,
                gfs_init, gfs_run_fileop, gfs_run_gread, gfs_run_gwrite, gfs_run_randread, gfs_run_seqread,
                gfs_shutdown, gfs_stats, gfs_device_ctx)
 
@@ -63,6 +63,16 @@ class GpuFS:
 
     def info(self) -> dict:
         return gfs_info(self.h)
+
+    # peer caches (NEXT-1) -------------------------------------------------
+    def export(self) -> bytes:
+        """Describe this cache for attach_peer in another process or GpuFS (gfs_export)."""
+        return gfs_export(self.h)
+
+    def attach_peer(self, desc: bytes) -> int:
+        """Map another cache (its export()) as a read-only peer: misses of read-only
+        files are filled from it over NVLink when it holds the same version (gfs_attach_peer)."""
+        return gfs_attach_peer(self.h, desc)
 
     @property
     def ctx(self) -> int:

@@ -144,9 +144,10 @@ struct VersionTable {
     VEntry* x = find(dev, ino, false);
     return x ? __atomic_load_n(&x->version, __ATOMIC_ACQUIRE) : 0;
   }
-  void bump(uint64_t dev, uint64_t ino) {
+  // Returns the new version (0 if the table is unavailable).
+  uint64_t bump(uint64_t dev, uint64_t ino) {
     VEntry* x = find(dev, ino, true);
-    if (x) __atomic_fetch_add(&x->version, 1, __ATOMIC_ACQ_REL);
+    return x ? __atomic_fetch_add(&x->version, 1, __ATOMIC_ACQ_REL) + 1 : 0;
   }
 };
 
@@ -224,6 +225,8 @@ struct gfs_handle {
   size_t fd_cap = 1024;  // per worker
   VersionTable vt;
   std::atomic<uint64_t> hs[HS_N];
+  std::vector<gfs_peer> peers;   // views of other caches (gfs_attach_peer)
+  std::vector<void*> ipc_open;   // CUDA IPC mappings to close at shutdown
 };
 
 namespace {
@@ -632,7 +635,7 @@ uint8_t* hfid_wmap(gfs_handle* h, Worker& w, uint32_t id, int fd, uint64_t end) 
   return map;
 }
 
-int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
+int32_t do_write(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
   HostFile f;
   if (!hfid_meta(h, q.hfid, &f)) return -EBADF;
   if (!(f.mode & GFS_O_GWRONCE)) return -EBADF;  // read-only files are never written back
@@ -657,7 +660,9 @@ int32_t do_write(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   } else {
     h->hs[HS_MAPPED]++;
   }
-  h->vt.bump(f.dev, f.ino);
+  // the version this write-back left the file at: the GPU records it as the
+  // entry's synced version (peer fill); stored before completion
+  h->resp_h[slot].version = h->vt.bump(f.dev, f.ino);
   h->hs[HS_WRITE]++;
   h->hs[HS_BYTES_D2H] += q.len;
   return (int32_t)q.len;
@@ -723,7 +728,7 @@ void worker_loop(gfs_handle* h, int wi) {
     const auto tb = std::chrono::steady_clock::now();
     switch (q.op) {
       case GFS_OP_READ: res = do_read(h, w, q); break;
-      case GFS_OP_WRITE: res = do_write(h, w, q); break;
+      case GFS_OP_WRITE: res = do_write(h, w, slot, q); break;
       case GFS_OP_OPEN:
         res = do_open(h, w, slot, q);
         h->hs[HS_OPEN_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
@@ -762,9 +767,11 @@ void free_all(gfs_handle* h) {
   auto F = [](void* p) {
     if (p) cudaFree(p);
   };
+  for (void* p : h->ipc_open) cudaIpcCloseMemHandle(p);
+  h->ipc_open.clear();
   if (h->own_pool) F(h->h.pool);
   F(h->h.f_state); F(h->h.f_tag); F(h->h.f_file); F(h->h.f_valid); F(h->h.f_lo); F(h->h.f_hi);
-  F(h->h.f_written); F(h->h.f_stamp); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
+  F(h->h.f_written); F(h->h.f_stamp); F(h->h.f_hv); F((void*)h->h.peers); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
   F(h->h.node_free); F(h->h.node_free_top); F(h->h.node_lock); F(h->h.files); F(h->h.paths); F(h->h.uid_next);
   F(h->h.ack); F(h->h.ring_tail); F(h->h.ctr); F(h->h.staging_bits); F(h->d);
   if (h->ring_h) cudaFreeHost(h->ring_h);
@@ -861,6 +868,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMalloc((void**)&c.f_hi, nframes * 4));
   CK(cudaMalloc((void**)&c.f_written, nframes * 4));
   CK(cudaMalloc((void**)&c.f_stamp, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_hv, nframes * 4));
   CK(cudaMalloc((void**)&c.fresh_next, 4));
   CK(cudaMalloc((void**)&c.hand, 4));
   c.max_nodes = max_nodes;
@@ -965,6 +973,96 @@ GFS_API int gfs_shutdown(gfs_handle* h) {
 }
 
 GFS_API const gfs_ctx* gfs_device_ctx(gfs_handle* h) { return h ? h->d : nullptr; }
+
+// ------------------------------------------------------------------ peer caches (NEXT-1)
+namespace {
+constexpr uint64_t kExportMagic = 0x3152454550534647ull;  // "GFSPEER1"
+constexpr int kNExport = 7;  // pool, f_state, f_tag, f_lo, f_hv, nodes, files
+
+int push_ctx(gfs_handle* h) {
+  cudaSetDevice(h->cfg.device);
+  if (cudaMemcpyAsync(h->d, &h->h, sizeof(gfs_ctx), cudaMemcpyHostToDevice, h->priv) != cudaSuccess) return -EIO;
+  return cudaStreamSynchronize(h->priv) == cudaSuccess ? 0 : -EIO;
+}
+}  // namespace
+
+GFS_API int gfs_export(gfs_handle* h, gfs_export_desc* out) {
+  if (!h || !out) return -EINVAL;
+  if (!h->own_pool) return -ENOTSUP;  // IPC needs allocation bases; a caller-owned pool may be a sub-allocation
+  cudaSetDevice(h->cfg.device);
+  memset(out, 0, sizeof(*out));
+  out->magic = kExportMagic;
+  out->pid = (int32_t)getpid();
+  out->device = h->cfg.device;
+  out->page_shift = h->h.page_shift;
+  out->nframes = h->h.nframes;
+  out->max_nodes = h->h.max_nodes;
+  out->max_files = h->h.max_files;
+  const void* ptrs[kNExport] = {h->h.pool, h->h.f_state, h->h.f_tag, h->h.f_lo, h->h.f_hv, h->h.nodes, h->h.files};
+  for (int i = 0; i < kNExport; ++i) {
+    out->ptr[i] = (uint64_t)(uintptr_t)ptrs[i];
+    cudaIpcMemHandle_t m;
+    if (cudaIpcGetMemHandle(&m, (void*)ptrs[i]) != cudaSuccess) return -EIO;
+    static_assert(sizeof(m) == sizeof(out->ipc[0]), "IPC handle size");
+    memcpy(out->ipc[i], &m, sizeof(m));
+  }
+  if (!(h->h.flags & GFS_F_EXPORTED)) {  // fills publish at system scope from now on
+    h->h.flags |= GFS_F_EXPORTED;
+    const int r = push_ctx(h);
+    if (r) return r;
+  }
+  return 0;
+}
+
+GFS_API int gfs_attach_peer(gfs_handle* h, const gfs_export_desc* d) {
+  if (!h || !d || d->magic != kExportMagic) return -EINVAL;
+  if (d->page_shift != h->h.page_shift) return -EINVAL;  // frames are copied whole-page
+  if (d->nframes >= (1u << 27) || !d->max_files || (d->max_files & (d->max_files - 1))) return -EINVAL;
+  if (h->peers.size() >= GFS_MAX_PEERS) return -ENOSPC;
+  const bool local = d->pid == (int32_t)getpid();
+  if (local && d->ptr[0] == (uint64_t)(uintptr_t)h->h.pool) return -EINVAL;  // itself
+  cudaSetDevice(h->cfg.device);
+  void* p[kNExport] = {};
+  if (local) {
+    if (d->device != h->cfg.device) {
+      const cudaError_t e = cudaDeviceEnablePeerAccess(d->device, 0);
+      if (e != cudaSuccess && e != cudaErrorPeerAccessAlreadyEnabled) return -EIO;
+      cudaGetLastError();
+    }
+    for (int i = 0; i < kNExport; ++i) p[i] = (void*)(uintptr_t)d->ptr[i];
+  } else {
+    for (int i = 0; i < kNExport; ++i) {
+      cudaIpcMemHandle_t m;
+      memcpy(&m, d->ipc[i], sizeof(m));
+      if (cudaIpcOpenMemHandle(&p[i], m, cudaIpcMemLazyEnablePeerAccess) != cudaSuccess) {
+        fprintf(stderr, "gpufs: cudaIpcOpenMemHandle failed: %s\n", cudaGetErrorString(cudaGetLastError()));
+        for (int j = 0; j < i; ++j) cudaIpcCloseMemHandle(p[j]);
+        return -EIO;
+      }
+    }
+    for (int i = 0; i < kNExport; ++i) h->ipc_open.push_back(p[i]);
+  }
+  gfs_peer v{};
+  v.pool = (uint8_t*)p[0];
+  v.f_state = (uint64_t*)p[1];
+  v.f_tag = (uint64_t*)p[2];
+  v.f_lo = (uint32_t*)p[3];
+  v.f_hv = (uint32_t*)p[4];
+  v.nodes = (uint64_t*)p[5];
+  v.files = (gfs_file*)p[6];
+  v.nframes = d->nframes;
+  v.max_nodes = d->max_nodes;
+  v.max_files = d->max_files;
+  v.page_shift = d->page_shift;
+  h->peers.push_back(v);
+  if (!h->h.peers && cudaMalloc((void**)&h->h.peers, GFS_MAX_PEERS * sizeof(gfs_peer)) != cudaSuccess) return -ENOMEM;
+  if (cudaMemcpy((void*)h->h.peers, h->peers.data(), h->peers.size() * sizeof(gfs_peer), cudaMemcpyHostToDevice) !=
+      cudaSuccess)
+    return -EIO;
+  h->h.npeers = (uint32_t)h->peers.size();
+  const int r = push_ctx(h);
+  return r ? r : (int)h->peers.size() - 1;
+}
 
 GFS_API int gfs_stats(gfs_handle* h, uint64_t* out, int n, int reset) {
   if (!h || !out) return -EINVAL;

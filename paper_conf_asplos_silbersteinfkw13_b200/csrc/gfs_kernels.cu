@@ -33,6 +33,7 @@ __global__ void k_init_metadata(gfs_ctx c) {
     c.f_hi[i] = 0;
     c.f_written[i] = 0;
     c.f_stamp[i] = 0;
+    c.f_hv[i] = 0;
   }
   if (blockIdx.x == 0 && threadIdx.x == 0) {
     *c.fresh_next = 0;

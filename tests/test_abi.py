@@ -54,3 +54,22 @@ def test_init_without_gpu_fails_loudly():
     import paper_conf_asplos_silbersteinfkw13_b200 as g
     with pytest.raises(g.GfsError):
         g.gfs_init(g.gfs_config_default())
+
+
+def test_struct_layouts_match_the_header(tmp_path):
+    """ctypes mirrors of gfs_config / gfs_export_desc have the C sizes (gcc on include/gpufs.h)."""
+    import ctypes
+    import shutil
+    import subprocess
+    import paper_conf_asplos_silbersteinfkw13_b200 as g
+    if not shutil.which("gcc"):
+        pytest.skip("no gcc")
+    src = tmp_path / "sz.c"
+    src.write_text('#include <stdio.h>\n#include "gpufs.h"\nint main(void){printf("%zu %zu %zu\\n",'
+                   ' sizeof(gfs_config), sizeof(gfs_export_desc), sizeof(gfs_peer)); return 0;}\n')
+    exe = tmp_path / "sz"
+    subprocess.check_call(["gcc", "-I", os.path.join(ROOT, "include"), str(src), "-o", str(exe)])
+    cfg, desc, peer = map(int, subprocess.check_output([str(exe)]).split())
+    assert ctypes.sizeof(g.gfs_config) == cfg
+    assert ctypes.sizeof(g.gfs_export_desc) == desc
+    assert peer == 7 * 8 + 4 * 4
