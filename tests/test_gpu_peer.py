@@ -185,3 +185,57 @@ def test_peer_fill_across_processes_ipc(g, shmdir):
         open(done, "w").close()
         child.wait(timeout=120)
     assert child.returncode == 0
+
+
+def _c5_rank(rank, ws, port, root, size, iters, outdir):
+    """One rank of the C5 pipeline with peer caches (bench.py c5_phase at N = 2):
+    write f_r + gfsync, barrier, re-read f_{r+1} (first pass from the writer's
+    cache through CUDA IPC), barrier; both ranks share cuda:0 here."""
+    import socket  # noqa: F401
+    import torch
+    import torch.distributed as dist
+    import paper_conf_asplos_silbersteinfkw13_b200 as g
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=ws)
+    P = 1 << 21
+    mine, peer = f"{root}/f_{rank}.bin", f"{root}/f_{(rank + 1) % ws}.bin"
+    res = {"ok": True, "peer_fill": 0, "rpc_read": 0}
+    with g.GpuFS(cache_bytes=64 * P, page_size=P, daemon_threads=2, max_batch=8, timeout_ms=30000) as fs:
+        descs = [None] * ws
+        dist.all_gather_object(descs, fs.export())
+        for r, d in enumerate(descs):
+            if r != rank:
+                fs.attach_peer(d)
+        for it in range(iters):
+            data = np.random.default_rng(100 * it + rank).integers(0, 256, size=size, dtype=np.uint8)
+            src = torch.from_numpy(data).cuda()
+            res["ok"] &= fs.seqwrite(mine, src, chunk=P, grid=8, sync_grid=2) == 0
+            dist.barrier()
+            want = oracle.checksum(peer, 0, size)
+            for _ in range(2):
+                s, err = fs.seqread(peer, size, P, grid=8)
+                res["ok"] &= err == 0 and s == want
+            dist.barrier()
+        st = fs.stats()
+        res["peer_fill"], res["rpc_read"] = st["peer_fill"], st["rpc_read"]
+        dist.barrier()  # no rank unmaps a cache another still reads
+    with open(os.path.join(outdir, f"r{rank}.json"), "w") as f:
+        json.dump(res, f)
+    dist.destroy_process_group()
+
+
+def test_c5_world2_peer_pipeline(shmdir):
+    import socket
+    import torch.multiprocessing as mp
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    size, iters = 5 * (1 << 21) + 4096, 3
+    mp.spawn(_c5_rank, args=(2, port, shmdir, size, iters, shmdir), nprocs=2, join=True)
+    for r in range(2):
+        res = json.load(open(os.path.join(shmdir, f"r{r}.json")))
+        assert res["ok"], res
+        # every first re-read of an iteration comes from the writer's cache
+        assert res["peer_fill"] == iters * 6 and res["rpc_read"] == 0, res
