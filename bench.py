@@ -234,6 +234,34 @@ def run_ours(args):
     if int(res[1]) != 0:
         raise SystemExit(f"gread sweep error {int(res[1])}")
 
+    # K1 variant: the same sweep through gmmap/gmunmap (zero-copy
+    # mapping of each page; the consumer checksums the frame in place)
+    k1 = None
+    if not args.no_k1:
+        kt = []
+        last_path, last_sum = paths[(nstep[0] - 1) % 2], int(res[0]) & ((1 << 64) - 1)
+        k1_parity = True
+        with torch.cuda.stream(stream):
+            for rep in range(3):
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                out.zero_()
+                e0.record(stream)
+                fs.seqread(paths[nstep[0] % 2], size, P, use_mmap=True, grid=grid, stream=stream, sync=False,
+                           scratch=scratch, out=out)
+                e1.record(stream)
+                stream.synchronize()
+                if int(out[1].item()) != 0:
+                    raise SystemExit(f"gmmap sweep error {int(out[1].item())}")
+                if paths[nstep[0] % 2] == last_path:  # same file as the last gread sweep: same checksum
+                    k1_parity &= (int(out[0].item()) & ((1 << 64) - 1)) == last_sum
+                kt.append(e0.elapsed_time(e1))
+                nstep[0] += 1
+        k1_ms = float(np.median(kt))
+        k1 = {"workload": "K1: the C2 sweep through gmmap/gmunmap (one page mapped per call)",
+              "GBps": round(size / (k1_ms * 1e-3) / 1e9, 3), "ms": round(k1_ms, 3),
+              "frac_h2d": round(size / (k1_ms * 1e-3) / 1e9 / h2d, 4),
+              "checksum_matches_gread_sweep": bool(k1_parity)}
+
     # cache-hit phase (K4 shape): pre-warm a file that fits, random 16 KiB greads into smem
     hit = None
     if not args.no_hit:
@@ -293,6 +321,8 @@ def run_ours(args):
         line["c5"] = c5
     if fig4:
         line["fig4_page_sweep"] = fig4
+    if k1:
+        line["k1_gmmap"] = k1
     if not args.no_cpu:
         line["cpu_baseline"] = cpu_baseline(args, path, size)
     print(json.dumps(line), flush=True)
@@ -339,6 +369,15 @@ def hit_phase(args, torch, g, gen, fs_unused, dev, stream, hbm, rank):
                 run_r()
             ms_g = timed(run_g, 5)
             ms_r = timed(run_r, 5)
+            # K5 ablation (Table 2): the same calls, every lookup
+            # under the file lock, against lock-free lookups (fewer calls: the
+            # locked variant serialises every block on one file's lock)
+            abl_calls = 32
+            d_off_a = d_off[:grid * abl_calls]
+            run_a = lambda: fs.randread(path, chunk, d_off_a, grid, block=args.hit_block, stream=stream,
+                                        sync=False, out=out)
+            run_a()
+            ms_lockfree = timed(run_a, 3)
             out.zero_()
             run_g()
             stream.synchronize()
@@ -349,6 +388,17 @@ def hit_phase(args, torch, g, gen, fs_unused, dev, stream, hbm, rank):
             sr = int(out[0].item()) & ((1 << 64) - 1)
         st = fs.stats()
         del raw
+    ms_locked = None
+    with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, device=torch.cuda.current_device(),
+                 daemon_threads=args.daemon_threads, timeout_ms=args.timeout_ms, flags=g.F_LOCKED_TRAVERSAL) as fl:
+        s2, err2 = fl.seqread(path, size, P, grid=296)
+        assert err2 == 0 and s2 == s
+        with torch.cuda.stream(stream):
+            run_l = lambda: fl.randread(path, chunk, d_off_a, grid, block=args.hit_block, stream=stream,
+                                        sync=False, out=out)
+            run_l()
+            ms_locked = timed(run_l, 3)
+        stl = fl.stats()
     nbytes = grid * calls * chunk
     gbs = nbytes / (ms_g * 1e-3) / 1e9
     return {"workload": f"K4: {grid} blocks x {calls} x 16 KiB gread -> smem, random offsets, {args.hit_file_gib} GiB "
@@ -358,7 +408,13 @@ def hit_phase(args, torch, g, gen, fs_unused, dev, stream, hbm, rank):
             "roofline": {"bound": "hbm", "achieved": round(gbs, 3), "peak": hbm, "unit": "GB/s",
                          "frac": round(gbs / hbm, 4), "traffic": None,
                          "note": "1 algorithmic HBM byte per delivered byte (frame read; destination is smem)"},
-            "checksum_match_raw": sg == sr, "misses_after_warm": st["miss"], "ms": round(ms_g, 3)}
+            "checksum_match_raw": sg == sr, "misses_after_warm": st["miss"], "ms": round(ms_g, 3),
+            "k5_locked_ablation": {"calls_per_block": abl_calls, "lockfree_ms": round(ms_lockfree, 3),
+                                   "locked_ms": round(ms_locked, 3),
+                                   "lockfree_speedup": round(ms_locked / ms_lockfree, 2),
+                                   "locked_lookups": stl["locked"],
+                                   "note": "GFS_F_LOCKED_TRAVERSAL: every lookup takes the file lock (the paper "
+                                           "reports lock-free ~3x faster, P:L1047-1048)"}}
 
 
 def grep_phase(args, torch, g, gen, dev, stream, hbm, rank, ws, local, dist):
@@ -686,6 +742,7 @@ def main():
     ap.add_argument("--no-matvec", action="store_true")
     ap.add_argument("--no-c5", action="store_true")
     ap.add_argument("--no-fig4", action="store_true")
+    ap.add_argument("--no-k1", action="store_true")
     ap.add_argument("--c5-mib", type=int, default=512)
     ap.add_argument("--c5-iters", type=int, default=3)
     ap.add_argument("--c5-sync-grid", type=int, default=8)

@@ -461,6 +461,7 @@ struct ScanSmem {
   uint32_t* ccnt;
   uint16_t* olist;  // occupied count slots, in insertion order
   uint64_t hf;      // splitmix64(file index) of the current item (digest)
+  uint32_t cmask;   // count table slots - 1
 };
 
 // One hit of word k at file position pos: per-item shared count (spilling to
@@ -468,9 +469,9 @@ struct ScanSmem {
 __device__ __forceinline__ void count_hit(GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
                                           uint32_t f, uint32_t k, uint64_t pos, uint64_t* hits, uint64_t hit_cap,
                                           ScanAcc& acc) {
-  uint32_t cs = (k * 2654435761u) & (kCountSlots - 1);
+  uint32_t cs = (k * 2654435761u) & S.cmask;
   bool done = false;
-  for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & (kCountSlots - 1)) {
+  for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & S.cmask) {
     const uint32_t prev = atomicCAS(&S.ckey[cs], 0u, k + 1);
     if (prev == 0) S.olist[atomicAdd(nocc, 1u)] = (uint16_t)cs;
     if (prev == 0 || prev == k + 1) {
@@ -577,6 +578,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
   S.ckey = S.mask + ((nstripe_max + 1 + 3) & ~3u);
   S.ccnt = S.ckey + kCountSlots;
   S.olist = (uint16_t*)(S.ccnt + kCountSlots);
+  S.cmask = kCountSlots - 1;
   uint16_t* tok = S.olist + kCountSlots;  // token starts of one round: <= 32 per thread
   const uint32_t round_stripes = 2u * (uint32_t)nthr;
   __shared__ uint64_t nxt_item, nxt_size, nxt_base;
@@ -727,6 +729,156 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
     }
   }
   // block-level digest reduction
+  for (int o = 16; o; o >>= 1) {
+    acc.dsum += __shfl_xor_sync(0xFFFFFFFFu, acc.dsum, o);
+    acc.dxor ^= __shfl_xor_sync(0xFFFFFFFFu, acc.dxor, o);
+    acc.nh += __shfl_xor_sync(0xFFFFFFFFu, acc.nh, o);
+  }
+  if (lane == 0) {
+    atomicAdd(&w.vars[V_DSUM], (unsigned long long)acc.dsum);
+    atomicXor(&w.vars[V_DXOR], (unsigned long long)acc.dxor);
+    atomicAdd(&w.vars[V_NHITS], (unsigned long long)acc.nh);
+  }
+}
+
+// ------------------------------------------------------------ warp-item scan
+// The same method as k_grep_scan with one WARP per item (warp-collective
+// gread_warp, the paper's design point P:L256-271): no block barrier in the
+// item loop, so a warp waiting on its lookups or probes never holds up the
+// others. Items are smaller (the chunk, e.g. 8 KiB) so a warp's buffer, mask,
+// count table and token list fit in ~16 KiB of shared memory.
+constexpr uint32_t kWarpSlots = 256;  // per-warp count table (overflow spills to the global table)
+constexpr uint32_t kWarpTok = 2048;   // bytes: 64 stripes x <= 16 token starts x u16
+
+__host__ __device__ __forceinline__ uint32_t warp_region_bytes(uint32_t chunk) {
+  const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
+  const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
+  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + kWarpSlots * 8 + kWarpSlots * 2 + kWarpTok + 16;
+}
+
+__global__ void __launch_bounds__(256) k_grep_scan_warp(const gfs_ctx* c, GrepWork w, uint32_t chunk,
+                                                         uint64_t* hits, uint64_t hit_cap, uint64_t* totals,
+                                                         uint32_t* rec, uint64_t rec_cap) {
+  extern __shared__ __align__(16) uint8_t sm[];
+  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+  uint8_t* base = sm + (size_t)wid * warp_region_bytes(chunk);
+  const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
+  const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
+  ScanSmem S;
+  S.buf = base;
+  S.mask = (uint32_t*)(base + buf_bytes);
+  S.ckey = S.mask + ((nstripe_max + 1 + 3) & ~3u);
+  S.ccnt = S.ckey + kWarpSlots;
+  S.olist = (uint16_t*)(S.ccnt + kWarpSlots);
+  S.cmask = kWarpSlots - 1;
+  uint16_t* tok = S.olist + kWarpSlots;
+  uint32_t* wv = (uint32_t*)((uint8_t*)tok + kWarpTok);  // [0] occupied slots, [1] spilled
+  const uint64_t nitems = w.vars[V_NITEMS];
+  ScanAcc acc{0, 0, 0};
+  for (uint32_t i = lane; i < kWarpSlots; i += 32) {  // dynamic smem is not cleared between launches
+    S.ckey[i] = 0;
+    S.ccnt[i] = 0;
+  }
+  // lane 0 claims the next item; its fields are loaded by every lane (broadcast)
+  uint64_t item = 0;
+  if (lane == 0) item = atomicAdd(&w.vars[V_NEXT], 1ull);
+  item = __shfl_sync(0xFFFFFFFFu, item, 0);
+  while (item < nitems) {
+    const uint32_t f = w.item_file[item];
+    const int fd = w.fd[f];
+    const uint64_t size = w.size[f];
+    const uint64_t s = (item - w.item_base[f]) * chunk;
+    uint64_t next = 0;  // claimed now, so its fields' loads overlap this item
+    if (lane == 0) {
+      next = atomicAdd(&w.vars[V_NEXT], 1ull);
+      wv[0] = 0;
+      wv[1] = 0;
+    }
+    S.hf = splitmix64(f);
+    const uint64_t e = min(size, s + chunk);
+    const uint64_t ws = s >= kPre ? s - kPre : 0;
+    const uint64_t we = min(size, e + kHalo);
+    const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
+    const int64_t r = gread_warp(c, fd, ws, we - ws, S.buf + vlo);
+    next = __shfl_sync(0xFFFFFFFFu, next, 0);
+    if (r != (int64_t)(we - ws)) {
+      if (lane == 0) set_err(w, r < 0 ? r : -EIO);
+      item = next;
+      continue;
+    }
+    // pass 1: word-byte bits per 32-byte stripe; bytes outside [vlo, vhi) are non-word
+    const uint32_t nstripe = (vhi + 31) / 32;
+    for (uint32_t j = lane; j < nstripe; j += 32)
+      S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
+    if (lane == 0) S.mask[nstripe] = 0;
+    __syncwarp();
+    // pass 2, 64 stripes per round: token starts in [s, e) compacted into tok
+    const uint32_t olo = kPre, ohi = kPre + (uint32_t)(e - s);
+    const uint32_t jlo = olo / 32, jhi = (ohi - 1) / 32;
+    for (uint32_t r0 = jlo; r0 <= jhi; r0 += 64) {
+      uint32_t st[2];
+      uint32_t cnt = 0;
+#pragma unroll
+      for (int q = 0; q < 2; ++q) {
+        const uint32_t j = r0 + 2 * (uint32_t)lane + q;
+        st[q] = 0;
+        if (j <= jhi) {
+          const uint32_t m = S.mask[j];
+          const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
+          st[q] = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
+        }
+        cnt += __popc(st[q]);
+      }
+      uint32_t incl = cnt;
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+        if (lane >= o) incl += t;
+      }
+      const uint32_t total = __shfl_sync(0xFFFFFFFFu, incl, 31);
+      uint32_t off = incl - cnt;
+#pragma unroll
+      for (int q = 0; q < 2; ++q) {
+        const uint32_t jb = 32 * (r0 + 2 * (uint32_t)lane + q);
+        for (uint32_t x = st[q]; x; x &= x - 1) tok[off++] = (uint16_t)(jb + __ffs(x) - 1);
+      }
+      __syncwarp();
+      for (uint32_t q = lane; q < total; q += 32) {
+        const uint32_t i = tok[q], j = i >> 5, b = i & 31;
+        const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | S.mask[j];
+        const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
+        if (L <= 32)                                   // no dictionary word is longer (R12)
+          scan_token(w, S, &wv[0], &wv[1], f, i, L, s + i - kPre, hits, hit_cap, acc);
+      }
+      __syncwarp();  // tok is reused by the next round
+    }
+    // flush: a whole-file item with no spill owns its records; otherwise merge
+    const uint32_t nocc = wv[0];
+    const bool direct = s == 0 && e == size && !wv[1] && rec;
+    unsigned long long rbase = 0;
+    if (direct && lane == 0 && nocc) rbase = atomicAdd(&w.vars[V_NREC], (unsigned long long)nocc);
+    rbase = __shfl_sync(0xFFFFFFFFu, rbase, 0);
+    for (uint32_t q = lane; q < nocc; q += 32) {
+      const uint32_t cs = S.olist[q];
+      const uint32_t k = S.ckey[cs] - 1, cnt = S.ccnt[cs];
+      S.ckey[cs] = 0;
+      S.ccnt[cs] = 0;
+      if (direct) {
+        atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
+        const uint64_t idx = rbase + q;
+        if (idx < rec_cap) {
+          rec[3 * idx] = f;
+          rec[3 * idx + 1] = k;
+          rec[3 * idx + 2] = cnt;
+        } else {
+          set_err(w, -ENOSPC);
+        }
+      } else {
+        pair_add(w, f, k, cnt);
+      }
+    }
+    __syncwarp();  // count table and wv are reset before the next item uses them
+    item = next;
+  }
   for (int o = 16; o; o >>= 1) {
     acc.dsum += __shfl_xor_sync(0xFFFFFFFFu, acc.dsum, o);
     acc.dxor ^= __shfl_xor_sync(0xFFFFFFFFu, acc.dxor, o);
@@ -943,9 +1095,13 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   cudaEventRecord(ev, s);
 
   const gfs_ctx* c = gfs_device_ctx(h);
-  const uint32_t smem = scan_smem(p->chunk, p->block);
+  // GFS_GREP_WARP=1: one warp per item (k_grep_scan_warp)
+  const bool warp_items = getenv("GFS_GREP_WARP") && *getenv("GFS_GREP_WARP") == '1';
+  const uint32_t smem = warp_items ? warp_region_bytes(p->chunk) * (p->block / 32) : scan_smem(p->chunk, p->block);
   if (smem > 227 * 1024) return -EINVAL;
-  cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (warp_items && p->block / 32 > GFS_WARP_API_MAX_WARPS) return -EINVAL;
+  cudaFuncSetAttribute(warp_items ? (const void*)k_grep_scan_warp : (const void*)k_grep_scan,
+                       cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   // GFS_GREP_DEBUG=1: synchronise after each stage, print its time and the first error
   const bool dbg = getenv("GFS_GREP_DEBUG") && *getenv("GFS_GREP_DEBUG") == '1';
   static unsigned long long* d_prof = nullptr;
@@ -995,7 +1151,8 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
   // persistent scan grid: every resident block slot once (p->grid caps it)
   int occ = 1;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_scan, (int)p->block, smem);
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, warp_items ? (const void*)k_grep_scan_warp
+                                                                 : (const void*)k_grep_scan, (int)p->block, smem);
   // GFS_GREP_BPS=n: at most n scan blocks per SM, the rest of the SM's
   // L1/shared-memory array left to L1 (dictionary buckets of frequent words)
   if (getenv("GFS_GREP_BPS")) {
@@ -1005,8 +1162,12 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
     cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributePreferredSharedMemoryCarveout, pct < 100 ? pct : 100);
   }
   const uint32_t scan_grid = (uint32_t)(occ > 0 ? occ : 1) * (uint32_t)nsm;
-  k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
-      c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
+  if (warp_items)
+    k_grep_scan_warp<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
+        c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
+  else
+    k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
+        c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
   stage("scan");
   if (!p->keep_open) k_grep_close<<<nsm * 16, 32, 0, s>>>(c, w);
   k_grep_compact<<<nsm * 8, 256, 0, s>>>(w, d_rec, d_rec ? rec_cap : 0, d_totals);

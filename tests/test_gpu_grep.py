@@ -92,3 +92,15 @@ def test_cache_smaller_than_corpus(g, shmdir):
         st = fs.stats()
     compare(out, ref)
     assert st["evict"] > 0
+
+
+@pytest.mark.parametrize("chunk", [16, 4096])
+def test_warp_item_scan_vs_oracle(g, shmdir, chunk, monkeypatch):
+    """k_grep_scan_warp (one warp per item, gread_warp; GFS_GREP_WARP=1) is bit-exact too."""
+    monkeypatch.setenv("GFS_GREP_WARP", "1")
+    c = gen.c4_corpus(os.path.join(shmdir, "c4w"), seed=12, nfiles=300, total_bytes=3 << 20, nwords=2000)
+    ref = oracle.grep(c["dict"], c["list"], want_hits=True)
+    with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4,
+                 max_files=1024) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=True, chunk=chunk, grid=64)
+    compare(out, ref)
