@@ -162,6 +162,14 @@ int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, con
                      uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
                      int64_t* d_err, uint32_t grid, uint32_t block);
 
+/* The same benchmark with the warp-collective API (gread_warp):
+ * block/32 warps per block, each with its own `chunk` bytes of shared memory,
+ * warp w of block b issuing calls w, w + block/32, ... of block b's
+ * calls_per_block. block: a multiple of 32, at most 256. */
+int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
+                          uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
+                          int64_t* d_err, uint32_t grid, uint32_t block);
+
 /* Write harness: each block gopen(path, O_GWRONCE) and issues
  * d_ret[i] = gwrite(fd, d_off[i], d_len[i], d_src + d_srcoff[i]) for its calls,
  * then gclose. */

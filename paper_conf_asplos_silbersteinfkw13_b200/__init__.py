@@ -88,6 +88,7 @@ def lib():
             "gfs_run_gread": ([P, P, CS, I, U32, P, P, P, P, P, U32, U32, U32], I),
             "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
+            "gfs_run_randread_warp": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32], I),
             "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
             "gfs_run_seqwrite": ([P, P, CS, U64, U64, P, P, P, U32, U32, U32], I),
@@ -190,6 +191,12 @@ def gfs_run_seqread(h, stream, path, file_off, total, chunk, use_mmap, d_scratch
 def gfs_run_randread(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):
     return _ck(lib().gfs_run_randread(h, stream, _b(path) if path else None, raw, d_raw, chunk, calls_per_block,
                                       d_off, d_sum, d_err, grid, block), "gfs_run_randread")
+
+
+def gfs_run_randread_warp(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):
+    return _ck(lib().gfs_run_randread_warp(h, stream, _b(path) if path else None, raw, d_raw, chunk,
+                                           calls_per_block, d_off, d_sum, d_err, grid, block),
+               "gfs_run_randread_warp")
 
 
 def gfs_run_seqwrite(h, stream, path, total, chunk, d_src, d_err, d_tmp, grid, block, sync_grid):

@@ -151,7 +151,7 @@ class GpuFS:
         return int(out[0].item())
 
     # cache-hit reads into shared memory (K4) ---------------------------------
-    def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None):
+    def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None, warp=False):
         torch = _torch()
         dev = f"cuda:{self.device}"
         if isinstance(offs, torch.Tensor):
@@ -163,7 +163,9 @@ class GpuFS:
         if out is None:
             out = torch.zeros(2, dtype=torch.int64, device=dev)
         s, sp = self._stream(stream)
-        gfs_run_randread(self.h, sp, path, 1 if raw is not None else 0,
+        from . import gfs_run_randread_warp
+        fn = gfs_run_randread_warp if warp else gfs_run_randread
+        fn(self.h, sp, path, 1 if raw is not None else 0,
                          raw.data_ptr() if raw is not None else None, chunk, calls, d_off.data_ptr(),
                          out.data_ptr(), out.data_ptr() + 8, grid, block)
         if not sync:

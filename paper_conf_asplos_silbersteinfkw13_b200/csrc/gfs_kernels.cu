@@ -257,6 +257,59 @@ __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const cha
   if (!raw) gclose(c, fd);
 }
 
+// K4 with the warp-collective API (the paper's design point):
+// every warp issues its own gread_warp calls into its own chunk of shared
+// memory (warp w takes calls w, w + nwarps, ...), so one warp's lookup never
+// stalls the block's other warps at a barrier. raw: the same per-warp TMA
+// copies without GPUfs.
+__global__ void __launch_bounds__(256) k_randread_warp(const gfs_ctx* c, const char* path, int raw,
+                                                       const uint8_t* rawp, uint32_t chunk, uint32_t calls,
+                                                       const uint64_t* offs, uint64_t* sum, int64_t* err) {
+  extern __shared__ __align__(16) uint8_t smem[];
+  __shared__ uint64_t raw_mbar[GFS_WARP_API_MAX_WARPS];
+  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5, nw = blockDim.x >> 5;
+  uint8_t* buf = smem + (size_t)wid * chunk;
+  int fd = 0;
+  if (!raw) {
+    fd = gopen_warp(c, path, GFS_O_RDONLY);
+    if (fd < 0) {
+      if (lane == 0) note_err(err, fd);
+      return;
+    }
+  } else {
+    if (lane == 0) detail::mbar_init(&raw_mbar[wid]);
+    __syncwarp();
+  }
+  uint64_t s = 0;
+  uint32_t ph = 0;
+  const uint64_t* my = offs + (size_t)blockIdx.x * calls;
+  for (uint32_t i = wid; i < calls; i += nw) {
+    const uint64_t o = my[i];
+    int64_t r;
+    if (raw) {
+      __syncwarp();
+      if (lane == 0) {
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        detail::mbar_expect_tx(&raw_mbar[wid], chunk);
+        detail::tma_load(buf, rawp + o, chunk, &raw_mbar[wid]);
+      }
+      detail::mbar_wait(&raw_mbar[wid], ph);
+      ph ^= 1u;
+      r = chunk;
+    } else {
+      r = gread_warp(c, fd, o, chunk, buf);
+      if (r < 0) {
+        if (lane == 0) note_err(err, r);
+        break;
+      }
+    }
+    s += checksum_words(buf, o, (uint64_t)r, lane, 32, false);
+  }
+  s = warp_sum(s);
+  if (lane == 0) atomicAdd((unsigned long long*)sum, (unsigned long long)s);
+  if (!raw) gclose_warp(c, fd);
+}
+
 __global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
                                const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret) {
   const int fd = gopen(c, path, GFS_O_GWRONCE);
@@ -425,6 +478,22 @@ GFS_API int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int 
   if (chunk > 48 * 1024) cudaFuncSetAttribute(k_randread, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
   k_randread<<<grid, block, chunk, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
                                         d_off, d_sum, d_err);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
+                                  uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
+                                  int64_t* d_err, uint32_t grid, uint32_t block) {
+  if ((!raw && !h) || (raw && !d_raw) || grid == 0 || block == 0 || (block & 31) ||
+      block / 32 > GFS_WARP_API_MAX_WARPS || chunk == 0 || (chunk & 15) || (uint64_t)chunk * (block / 32) > 200 * 1024)
+    return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = raw ? nullptr : stage_path(path, s);
+  if (!raw && !dp) return -ENAMETOOLONG;
+  const uint32_t smem = chunk * (block / 32);
+  if (smem > 48 * 1024) cudaFuncSetAttribute(k_randread_warp, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  k_randread_warp<<<grid, block, smem, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk,
+                                             calls_per_block, d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
 

@@ -194,6 +194,11 @@ def test_randread_smem_checksum(g, shmdir):
         raw = torch.as_tensor(np.fromfile(path, dtype=np.uint8), device="cuda")
         s3, _ = fs.randread(None, chunk, offs, grid, raw=raw)
         assert s3 == expect
+        # warp-collective variant (gread_warp per warp, 4 warps per block), and its raw baseline
+        s4, err4 = fs.randread(path, chunk, offs, grid, block=128, warp=True)
+        assert err4 == 0 and s4 == expect
+        s5, _ = fs.randread(None, chunk, offs, grid, block=128, raw=raw, warp=True)
+        assert s5 == expect
     assert st["miss"] <= 256
 
 
