@@ -137,7 +137,9 @@ int gfs_info(gfs_handle* h, uint64_t* out, int n);
  *           into global memory. block: a multiple of 32, at most
  *           32 * GFS_WARP_API_MAX_WARPS (256).
  *   mode 5: like mode 4 into the warp's own shared buffer of smem_bytes
- *           (co-aligned at d_off[i] % 16), copied out afterwards. If gopen fails every d_ret[i] of that block gets its error. */
+ *           (co-aligned at d_off[i] % 16), copied out afterwards. If gopen fails every d_ret[i] of that block gets its error.
+ * Bits 8+ of mode: the open flags of modes 0-3 (GFS_O_RDONLY, or GFS_O_RDWR to read
+ * a file the GPU also writes); modes 4-5 open read-only. */
 int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
                   const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
                   int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes);
@@ -170,12 +172,22 @@ int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path, int raw
                           uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
                           int64_t* d_err, uint32_t grid, uint32_t block);
 
-/* Write harness: each block gopen(path, O_GWRONCE) and issues
+/* Write harness: each block gopen(path, flags) — GFS_O_GWRONCE (write-once,
+ * diff against zeros) or GFS_O_RDWR (pages fetched, diff against
+ * a pristine copy) — and issues
  * d_ret[i] = gwrite(fd, d_off[i], d_len[i], d_src + d_srcoff[i]) for its calls,
- * then gclose. */
+ * then gclose. -EINVAL for other flags. */
 int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncalls, const uint64_t* d_off,
                    const uint64_t* d_len, const uint64_t* d_srcoff, const uint8_t* d_src, int64_t* d_ret,
-                   uint32_t grid, uint32_t block);
+                   uint32_t grid, uint32_t block, int flags);
+
+/* Writable-mapping harness (O_RDWR, Tab.1 gmmap/gmsync): block b
+ * takes calls b, b + grid, ...: gmmap(d_off[i], d_len[i], GFS_PROT_WRITE), store
+ * d_src + d_srcoff[i] through the pointer (the mapped prefix only), gmsync the
+ * page if do_msync, gmunmap. d_ret[i] = bytes mapped or -errno. */
+int gfs_run_mmap_write(gfs_handle* h, void* stream, const char* path, uint32_t ncalls, const uint64_t* d_off,
+                       const uint64_t* d_len, const uint64_t* d_srcoff, const uint8_t* d_src, int64_t* d_ret,
+                       uint32_t grid, uint32_t block, int do_msync);
 
 /* One-block file operations: op 0 = gfsync, 1 = gftruncate(arg), 2 = gfstat_size,
  * 3 = gopen+gclose only, 4 = pin (gopen without gclose: the file stays open

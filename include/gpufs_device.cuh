@@ -706,6 +706,7 @@ __device__ __forceinline__ uint32_t frame_init(const gfs_ctx* c, uint32_t f, uin
   st_rlx(&c->f_hi[f], 0);
   st_rlx(&c->f_written[f], 0);
   st_rlx(&c->f_hv[f], 0);
+  st_rlx(&c->f_pristine[f], 0);
   st_rlx(&c->f_stamp[f], stamp_now());
   // EVICTING -> FILLING|1 and generation + 1 as one atomic delta: readers that
   // found the frame through a stale slot may hold transient +1s they are about
@@ -725,6 +726,25 @@ __device__ __forceinline__ void synced(const gfs_ctx* c, uint32_t f, uint32_t lo
   if (fi < c->max_files) atomicMax((unsigned long long*)&c->files[fi].synced_version, (unsigned long long)version);
 }
 
+// Drop the page a published frame holds: tag cleared, generation + 1 (every
+// tree slot naming the old generation is now stale), `flag` (held by the
+// caller) cleared, in one atomic delta.
+__device__ __forceinline__ void frame_retire(const gfs_ctx* c, uint32_t f, uint32_t flag) {
+  st_rlx64(&c->f_tag[f], GFS_TAG_NONE);
+  a64_add_rel(&c->f_state[f], (1ull << 32) - (uint64_t)flag);
+}
+
+// O_RDWR: drop frame f's pristine copy (after its diff was
+// written back). The pristine frame was held FILLING|1 (never evictable).
+__device__ __forceinline__ void pristine_free(const gfs_ctx* c, uint32_t f) {
+  const uint32_t pv = ld_rlx(&c->f_pristine[f]);
+  if (pv == 0 || pv == GFS_PRISTINE_PENDING) return;
+  st_rlx(&c->f_pristine[f], 0);
+  const uint32_t pf = pv - 1;
+  frame_retire(c, pf, GFS_ST_FILLING);   // generation + 1, tag none
+  a64_add_rel(&c->f_state[pf], kRefDec);  // unreferenced: reclaimable (tier 0)
+}
+
 // Write back a frame's dirty range from one thread (the caller owns the frame:
 // EVICTING, ref 0): copy it into a staging slot over PCIe, then WRITE RPC.
 __device__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
@@ -733,17 +753,39 @@ __device__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t h
   const uint32_t hi = ld_rlx(&c->f_hi[f]);
   const uint32_t wr = ld_rlx(&c->f_written[f]);
   const uint64_t page = ld_rlx64(&c->f_tag[f]) & 0xFFFFFFFFull;
-  const int st = stage_alloc(c);
-  if (st < 0) return st;
+  const uint32_t pv = ld_rlx(&c->f_pristine[f]);
+  const bool diff = pv != 0 && pv != GFS_PRISTINE_PENDING;  // O_RDWR page: diff against its pristine copy
+  int st = -1, st2 = -1;
+  const uint64_t t0 = now_ns();
+  for (uint32_t ns = 64;;) {  // both slots or none: never wait for one while holding the other
+    st = stage_alloc(c, false);
+    if (st >= 0 && diff) {
+      st2 = stage_alloc(c, false);
+      if (st2 < 0) {
+        stage_free(c, st);
+        st = -1;
+      }
+    }
+    if (st >= 0) break;
+    backoff(ns);
+    if (timed_out(c, t0)) return -ETIMEDOUT;
+  }
   // frame bytes via L2 (.cg): this SM's L1 may hold lines of a previous tenant
   block_copy_from_frame(stage_ptr(c, st) + lo, frame_ptr(c, f) + lo, hi - lo, 0, 1);
+  if (diff) block_copy_from_frame(stage_ptr(c, st2) + lo, frame_ptr(c, pv - 1) + lo, hi - lo, 0, 1);
   __threadfence_system();
   gfs_rpc_resp rs;
   const int32_t r = rpc_call(c, GFS_OP_WRITE, hfid, (page << c->page_shift) + lo, st, hi - lo,
-                             wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, &rs);
+                             diff ? GFS_WF_DIFF : (wr >= hi - lo ? GFS_WF_FULL : 0u), diff ? (uint64_t)st2 : 0,
+                             nullptr, 0, &rs);
   stage_free(c, st);
+  if (st2 >= 0) stage_free(c, st2);
   if (r < 0) return r;
   synced(c, f, lo, hi, wr, rs.version);
+  if (diff) {
+    st_rlx(&c->f_hv[f], 0);
+    pristine_free(c, f);
+  }
   st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
   st_rlx(&c->f_hi[f], 0);
   st_rlx(&c->f_written[f], 0);
@@ -840,13 +882,6 @@ __device__ __forceinline__ void frame_release_rel(const gfs_ctx* c, uint32_t f) 
   a64_add_rel(&c->f_state[f], kRefDec);
 }
 
-// Drop the page a published frame holds: tag cleared, generation + 1 (every
-// tree slot naming the old generation is now stale), `flag` (held by the
-// caller) cleared, in one atomic delta.
-__device__ __forceinline__ void frame_retire(const gfs_ctx* c, uint32_t f, uint32_t flag) {
-  st_rlx64(&c->f_tag[f], GFS_TAG_NONE);
-  a64_add_rel(&c->f_state[f], (1ull << 32) - (uint64_t)flag);
-}
 
 // Give back a frame we installed but could not publish (lost the CAS race).
 __device__ __forceinline__ void frame_abandon(const gfs_ctx* c, uint32_t f) {
@@ -946,7 +981,9 @@ __device__ int peer_take(const gfs_ctx* c, const FileSnap& fs, uint64_t page, ui
       if (ld_rlx_sys64(&e->path_hash) != h || ld_rlx_sys(&e->path_len) != n) continue;
       if (ld_rlx_sys64(&e->ino) != ino || ld_rlx_sys64(&e->dev) != dev) continue;
       const uint32_t uid = ld_rlx_sys(&e->uid);
-      const bool wonce = (ld_rlx_sys(&e->oflags) & GFS_O_GWRONCE) != 0;
+      const uint32_t pof = ld_rlx_sys(&e->oflags);
+      if (pof & GFS_O_RDWR) break;  // a read-write peer's frames may hold unsynced or diffed bytes
+      const bool wonce = (pof & GFS_O_GWRONCE) != 0;
       const uint64_t ev = wonce ? ld_rlx_sys64(&e->synced_version) : ld_rlx_sys64(&e->version);
       if ((wonce && ev == 0) || ev != ver) break;  // the peer's copy is of another version
       if (!wonce && (ld_rlx_sys64(&e->size) != fs.size || (int64_t)ld_rlx_sys64((const uint64_t*)&e->mtime_ns) != mt))
@@ -1195,9 +1232,13 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
     }
     if (pull) {  // fill the frames this block installed: staging -> frame over PCIe, or peer frame -> frame
       for (uint32_t i = 0; i < cnt; ++i)
-        if (sc.frame[i] >= 0 && sc.fill[i] && sc.stage[i] != -1)
+        if (sc.frame[i] >= 0 && sc.fill[i] && sc.stage[i] != -1) {
           block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), fill_src(c, sc.stage[i]), sc.nbytes[i],
                                       tid, nthr);
+          // a writable page past the old EOF reads (and diffs) as zeros, not a previous tenant's bytes
+          if ((fs.oflags & GFS_O_RDWR) && sc.nbytes[i] < c->page_size)
+            block_zero(frame_ptr(c, (uint32_t)sc.frame[i]) + sc.nbytes[i], c->page_size - sc.nbytes[i], tid, nthr);
+        }
       if (c->flags & GFS_F_EXPORTED) __threadfence_system();  // peers read our frames at system scope
       else __threadfence();
       G::sync();
@@ -1236,6 +1277,57 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
       G::sync();
     }
   }
+}
+
+// O_RDWR: before the first local write to a page, preserve its
+// pristine copy. Block-collective over the held frames sc.frame[0, cnt): lane
+// i claims the pristine slot of page i (CAS 0 -> PENDING), allocates a frame
+// for it (held FILLING|1, so never evicted or found), the block copies the
+// working page into it and the lane publishes it; a page whose pristine copy
+// another block is making is waited for (that block only copies a frame it
+// holds: it never waits on us). Returns 0 or -errno (then no claim is left).
+template <class G = BlockGroup>
+__device__ int ensure_pristine(const gfs_ctx* c, Scratch& sc, uint32_t fdx, uint32_t cnt) {
+  const int tid = G::tid(), nthr = G::nthr();
+  if (tid == 0) sc.err = 0;
+  if (tid < (int)cnt) {
+    const uint32_t f = (uint32_t)sc.frame[tid];
+    sc.lo[tid] = GFS_DIRTY_NONE;  // pristine frame this lane must fill
+    if (ld_acq(&c->f_pristine[f]) == 0 && atom_cas(&c->f_pristine[f], 0u, GFS_PRISTINE_PENDING) == 0u) {
+      uint32_t gen = 0;
+      const int pf = alloc_frame(c, GFS_TAG_NONE, fdx, &gen);
+      if (pf < 0) {
+        st_rel(&c->f_pristine[f], 0u);
+        atomicMin(&sc.err, pf);
+      } else {
+        sc.lo[tid] = (uint32_t)pf;
+      }
+    }
+  }
+  G::sync();
+  for (uint32_t i = 0; i < cnt; ++i)
+    if (sc.lo[i] != GFS_DIRTY_NONE)
+      block_copy_from_frame(frame_ptr(c, sc.lo[i]), frame_ptr(c, (uint32_t)sc.frame[i]), c->page_size, tid, nthr);
+  __threadfence();
+  G::sync();
+  if (tid < (int)cnt) {
+    const uint32_t f = (uint32_t)sc.frame[tid];
+    if (sc.lo[tid] != GFS_DIRTY_NONE) {
+      st_rel(&c->f_pristine[f], sc.lo[tid] + 1u);
+    } else {
+      uint32_t ns = 64;
+      const uint64_t t0 = now_ns();
+      while (ld_acq(&c->f_pristine[f]) == GFS_PRISTINE_PENDING) {
+        backoff(ns);
+        if (timed_out(c, t0)) {
+          atomicMin(&sc.err, -ETIMEDOUT);
+          break;
+        }
+      }
+    }
+  }
+  G::sync();
+  return sc.err;
 }
 
 // ------------------------------------------------------------------ file table
@@ -1371,6 +1463,7 @@ __device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uin
       st_rlx(&c->f_hi[f], 0);
       st_rlx(&c->f_written[f], 0);
       st_rlx(&c->f_hv[f], 0);
+      pristine_free(c, f);
       frame_retire(c, f, GFS_ST_EVICTING);  // slots naming this generation go stale
     } else {
       a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
@@ -1417,7 +1510,7 @@ __device__ int new_incarnation(const gfs_ctx* c, gfs_file* e, uint32_t flags, co
   const uint64_t P = c->page_size;
   const uint64_t npages = ((uint64_t)rs.size + P - 1) >> c->page_shift;
   e->root = root;
-  e->height = (flags & GFS_O_GWRONCE) ? GFS_MAX_HEIGHT : height_for(npages);
+  e->height = (flags & GFS_O_WRITABLE) ? GFS_MAX_HEIGHT : height_for(npages);  // writable files grow
   e->uid = atomicAdd(c->uid_next, 1u);
   e->hfid = rs.hfid;
   e->size = (uint64_t)rs.size;
@@ -1452,7 +1545,7 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, uint32_t n, uint6
   pf->stage = -1;
   const bool want_pf = (flags_in & (int)GFS_O_PREFETCH) != 0;
   const int flags = flags_in & ~(int)GFS_O_PREFETCH;
-  if (flags != (int)GFS_O_RDONLY && flags != (int)GFS_O_GWRONCE) return -EINVAL;
+  if (flags != (int)GFS_O_RDONLY && flags != (int)GFS_O_GWRONCE && flags != (int)GFS_O_RDWR) return -EINVAL;
   if (n == 0) return -ENOENT;
   if (n >= GFS_MAX_PATH) return -ENAMETOOLONG;
   const uint32_t mask = c->max_files - 1;
@@ -1557,7 +1650,7 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, uint32_t n, uint6
       FileSnap old;
       old.fdx = i; old.uid = e->uid; old.root = e->root; old.height = e->height;
       old.hfid = e->hfid; old.oflags = e->oflags; old.size = e->size;
-      if (old.oflags & GFS_O_GWRONCE) {  // never lose written data: sync before dropping
+      if (old.oflags & GFS_O_WRITABLE) {  // never lose written data: sync before dropping
         const uint64_t np = (old.size + c->page_size - 1) >> c->page_shift;
         int r = sync_pages_lane(c, old, 0, np);
         if (r < 0 && r != -EBUSY) {
@@ -1639,7 +1732,7 @@ __device__ inline int gopen_t(const gfs_ctx* c, const char* path, int flags) {
     sc.stage[0] = pf.stage;
     sc.nbytes[0] = pf.nbytes;
     sc.cached_fd = -1;
-    if (fd >= 0 && detail::snap_fd(c, fd, &sc.cached) && !(sc.cached.oflags & GFS_O_GWRONCE)) {
+    if (fd >= 0 && detail::snap_fd(c, fd, &sc.cached) && !(sc.cached.oflags & GFS_O_WRITABLE)) {
       sc.cached_grid = detail::grid_id();
       sc.cached_blk = G::key();
       sc.cached_fd = fd;
@@ -1870,7 +1963,7 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
   __syncthreads();
   if (tid == 0) {
     FileSnap s;
-    if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_GWRONCE)) {
+    if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_WRITABLE)) {
       sc.ret = -EBADF;
     } else if (off + len < off || ((off + len) >> c->page_shift) >= (1ull << 32)) {
       sc.ret = -EINVAL;
@@ -1893,12 +1986,29 @@ __device__ inline int64_t gwrite(const gfs_ctx* c, int fd, uint64_t off, uint64_
     const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
     const int err = acquire_batch(c, sc, fs, pb, cnt, false);
     if (err) return err;
+    if (fs.oflags & GFS_O_RDWR) {
+      // pages past the host EOF start as zeros; then every page keeps its
+      // pristine copy before the first local write (diff-and-merge)
+      for (uint32_t i = 0; i < cnt; ++i)
+        if (sc.fill[i]) block_zero(frame_ptr(c, (uint32_t)sc.frame[i]), P, tid, nthr);
+      __syncthreads();
+      const int perr = ensure_pristine(c, sc, fs.fdx, cnt);
+      if (perr) {
+        if (tid < (int)cnt) {
+          const uint32_t f = (uint32_t)sc.frame[tid];
+          if (sc.fill[tid]) frame_retire(c, f, GFS_ST_FILLING);
+          frame_release(c, f);
+        }
+        __syncthreads();
+        return perr;
+      }
+    }
     for (uint32_t i = 0; i < cnt; ++i) {
       const uint64_t p = pb + i;
       const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
       const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
       uint8_t* fp = frame_ptr(c, (uint32_t)sc.frame[i]);
-      if (sc.fill[i]) {  // pristine copy is zeros
+      if (sc.fill[i] && !(fs.oflags & GFS_O_RDWR)) {  // pristine copy is zeros
         block_zero(fp, s, tid, nthr);
         block_zero(fp + e, P - e, tid, nthr);
       }
@@ -1947,7 +2057,7 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
   __syncthreads();
   if (sc.ret < 0) return (int)sc.ret;
   const FileSnap fs = sc.fs;
-  if (fs.oflags & GFS_O_GWRONCE) {
+  if (fs.oflags & GFS_O_WRITABLE) {
     const uint64_t np = (fs.size + c->page_size - 1) >> c->page_shift;
     const uint32_t B = nthr < 32 ? (uint32_t)nthr : 32u;
     uint32_t ns = 256;
@@ -1964,11 +2074,22 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
         if (f >= 0) {
           sc.lo[tid] = ld_rlx(&c->f_lo[f]);
           sc.hi[tid] = ld_rlx(&c->f_hi[f]);
+          const uint32_t pv = ld_rlx(&c->f_pristine[f]);
+          sc.nbytes[tid] = (pv != 0 && pv != GFS_PRISTINE_PENDING) ? pv : 0u;  // O_RDWR: pristine frame + 1
           // no waiting for a staging slot while holding a claimed page (other
           // blocks may hold the slots and wait for pages): give the claim
-          // back and redo this batch after the others are written
-          const int st = stage_alloc(c, false);
+          // back and redo this batch after the others are written. An O_RDWR
+          // page needs two slots (working and pristine ranges, GFS_WF_DIFF).
+          int st = stage_alloc(c, false), st2 = -1;
+          if (st >= 0 && sc.nbytes[tid]) {
+            st2 = stage_alloc(c, false);
+            if (st2 < 0) {
+              stage_free(c, st);
+              st = -1;
+            }
+          }
           sc.stage[tid] = st;
+          sc.fill[tid] = (uint32_t)st2;
           if (st < 0) {
             a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
             sc.frame[tid] = -1;
@@ -1978,23 +2099,34 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
       }
       __syncthreads();
       for (uint32_t i = 0; i < cnt; ++i)
-        if (sc.frame[i] >= 0)
+        if (sc.frame[i] >= 0) {
           block_copy_from_frame(stage_ptr(c, sc.stage[i]) + sc.lo[i], frame_ptr(c, (uint32_t)sc.frame[i]) + sc.lo[i],
-                           sc.hi[i] - sc.lo[i], tid, nthr);
+                                sc.hi[i] - sc.lo[i], tid, nthr);
+          if (sc.nbytes[i])
+            block_copy_from_frame(stage_ptr(c, (int)sc.fill[i]) + sc.lo[i], frame_ptr(c, sc.nbytes[i] - 1) + sc.lo[i],
+                                  sc.hi[i] - sc.lo[i], tid, nthr);
+        }
       __threadfence_system();
       __syncthreads();
       if (tid < (int)cnt && sc.frame[tid] >= 0) {
         const uint32_t f = (uint32_t)sc.frame[tid];
         const uint32_t lo = sc.lo[tid], hi = sc.hi[tid];
         const uint32_t wr = ld_rlx(&c->f_written[f]);
+        const bool diff = sc.nbytes[tid] != 0;
         gfs_rpc_resp rs;
         const int32_t r = rpc_call(c, GFS_OP_WRITE, fs.hfid, ((pb + tid) << c->page_shift) + lo, sc.stage[tid],
-                                   hi - lo, wr >= hi - lo ? GFS_WF_FULL : 0u, 0, nullptr, 0, &rs);
+                                   hi - lo, diff ? GFS_WF_DIFF : (wr >= hi - lo ? GFS_WF_FULL : 0u),
+                                   diff ? (uint64_t)sc.fill[tid] : 0, nullptr, 0, &rs);
         stage_free(c, sc.stage[tid]);
+        if (diff) stage_free(c, (int)sc.fill[tid]);
         if (r < 0) {
           atomicMin(&sc.err, r);
         } else {
           synced(c, f, lo, hi, wr, rs.version);
+          if (diff) {
+            st_rlx(&c->f_hv[f], 0);
+            pristine_free(c, f);
+          }
           st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
           st_rlx(&c->f_hi[f], 0);
           st_rlx(&c->f_written[f], 0);
@@ -2029,18 +2161,18 @@ __device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int pr
                               uint64_t* mapped_len) {
   using namespace detail;
   (void)addr;
-  (void)prot;
   (void)flags;
   Scratch& sc = scratch();
   const int tid = block_tid();
+  const bool wmap = (prot & (int)GFS_PROT_WRITE) != 0;
   __syncthreads();
   if (tid == 0) {
     FileSnap s;
     sc.ptr = nullptr;
     sc.aux = 0;
     sc.ret = 0;
-    if (!snap_fd_cached(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE)) {
-      sc.aux = -EBADF;
+    if (!snap_fd_cached(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE) || (wmap && !(s.oflags & GFS_O_RDWR))) {
+      sc.aux = -EBADF;  // a writable mapping needs an O_RDWR file
     } else if (off < s.size && len > 0) {
       sc.fs = s;
       sc.lc_ok = (sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id()) ? 1u : 0u;
@@ -2050,7 +2182,23 @@ __device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int pr
   __syncthreads();
   if (sc.ret == 1) {
     const FileSnap fs = sc.fs;
-    const int err = acquire_batch(c, sc, fs, off >> c->page_shift, 1, false);
+    int err = acquire_batch(c, sc, fs, off >> c->page_shift, 1, false);
+    if (!err && wmap) {  // writes through the pointer are untracked: keep the pristine copy, mark the range dirty
+      err = ensure_pristine(c, sc, fs.fdx, 1);
+      if (tid == 0) {
+        if (err) {
+          frame_release(c, (uint32_t)sc.frame[0]);
+        } else {
+          const uint32_t f = (uint32_t)sc.frame[0];
+          const uint64_t in = off & (c->page_size - 1);
+          uint64_t m = c->page_size - in;
+          if (len < m) m = len;
+          if (fs.size - off < m) m = fs.size - off;
+          atomicMin(&c->f_lo[f], (uint32_t)in);
+          atomicMax(&c->f_hi[f], (uint32_t)(in + m));
+        }
+      }
+    }
     if (tid == 0) {
       if (err) {
         sc.aux = err;
@@ -2089,6 +2237,110 @@ __device__ inline int gmunmap(const gfs_ctx* c, void* addr, uint64_t len) {
   return (int)sc.ret;
 }
 
+// gmsync: write back the dirty page mapped at `addr` now (Tab.1), for a
+// mapping the calling block holds (gmmap with GFS_PROT_WRITE on an O_RDWR
+// file). Only the bytes that differ from the page's pristine copy go to the
+// host (diff-and-merge); the pristine copy then becomes the
+// written-back state, so a later sync sends only later changes. The
+// application coordinates gmsync with other blocks' updates (Tab.1). Returns
+// 0, -EINVAL (not a mapped frame), -EBUSY (page being filled/evicted), or an
+// RPC error.
+__device__ inline int gmsync(const gfs_ctx* c, void* addr, uint64_t len, int flags) {
+  using namespace detail;
+  (void)len;
+  (void)flags;
+  Scratch& sc = scratch();
+  const int tid = block_tid(), nthr = block_nthr();
+  __syncthreads();
+  if (tid == 0) {
+    sc.ret = 0;
+    sc.frame[0] = -1;
+    const uint8_t* p = (const uint8_t*)addr;
+    if (p < c->pool || p >= c->pool + ((size_t)c->nframes << c->page_shift)) {
+      sc.ret = -EINVAL;
+    } else {
+      const uint32_t f = (uint32_t)((size_t)(p - c->pool) >> c->page_shift);
+      // claim: the caller's mapping holds a reference; EVICTING keeps other
+      // syncs and evictions off the page while its ranges are copied
+      uint64_t v = ld_rlx64(&c->f_state[f]);
+      for (;;) {
+        if (((uint32_t)v & GFS_ST_REF_MASK) == 0) {
+          sc.ret = -EINVAL;
+          break;
+        }
+        if ((uint32_t)v & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR)) {
+          sc.ret = -EBUSY;
+          break;
+        }
+        const uint64_t o = a64_cas(&c->f_state[f], v, v | GFS_ST_EVICTING);
+        if (o == v) break;
+        v = o;
+      }
+      if (sc.ret == 0) {
+        const uint32_t lo = ld_rlx(&c->f_lo[f]), pv = ld_rlx(&c->f_pristine[f]);
+        if (lo == GFS_DIRTY_NONE || pv == 0 || pv == GFS_PRISTINE_PENDING) {
+          a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));  // nothing written through a mapping
+        } else {
+          sc.frame[0] = (int)f;
+          sc.lo[0] = lo;
+          sc.hi[0] = ld_rlx(&c->f_hi[f]);
+          sc.nbytes[0] = pv;
+          sc.stage[0] = -1;
+          sc.fill[0] = 0xFFFFFFFFu;
+          const uint64_t t0 = now_ns();
+          for (uint32_t ns = 64;;) {  // both staging slots or none
+            const int a = stage_alloc(c, false);
+            const int b = a >= 0 ? stage_alloc(c, false) : -1;
+            if (b >= 0) {
+              sc.stage[0] = a;
+              sc.fill[0] = (uint32_t)b;
+              break;
+            }
+            if (a >= 0) stage_free(c, a);
+            backoff(ns);
+            if (timed_out(c, t0)) {
+              sc.ret = -ETIMEDOUT;
+              a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
+              sc.frame[0] = -1;
+              break;
+            }
+          }
+        }
+      }
+    }
+  }
+  __syncthreads();
+  if (sc.frame[0] < 0) return (int)sc.ret;
+  const uint32_t f = (uint32_t)sc.frame[0], lo = sc.lo[0], hi = sc.hi[0], pf = sc.nbytes[0] - 1;
+  block_copy_from_frame(stage_ptr(c, sc.stage[0]) + lo, frame_ptr(c, f) + lo, hi - lo, tid, nthr);
+  block_copy_from_frame(stage_ptr(c, (int)sc.fill[0]) + lo, frame_ptr(c, pf) + lo, hi - lo, tid, nthr);
+  __threadfence_system();
+  __syncthreads();
+  if (tid == 0) {
+    const uint64_t page = ld_rlx64(&c->f_tag[f]) & 0xFFFFFFFFull;
+    const uint32_t fi = ld_rlx(&c->f_file[f]);
+    gfs_rpc_resp rs;
+    const int32_t r = rpc_call(c, GFS_OP_WRITE, ld_rlx(&c->files[fi].hfid), (page << c->page_shift) + lo,
+                               sc.stage[0], hi - lo, GFS_WF_DIFF, (uint64_t)sc.fill[0], nullptr, 0, &rs);
+    stage_free(c, sc.stage[0]);
+    stage_free(c, (int)sc.fill[0]);
+    sc.ret = r < 0 ? r : 0;
+    if (r >= 0) {
+      ctr(c, GFS_C_WRITEBACK);
+      ctr(c, GFS_C_RPC_WRITE);
+      ctr(c, GFS_C_BYTES_D2H, hi - lo);
+    }
+  }
+  __syncthreads();
+  if (sc.ret == 0)  // the written-back state is the new pristine copy
+    block_copy_from_frame(frame_ptr(c, pf) + lo, frame_ptr(c, f) + lo, hi - lo, tid, nthr);
+  __threadfence();
+  __syncthreads();
+  if (tid == 0) a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
+  __syncthreads();
+  return (int)sc.ret;
+}
+
 // gftruncate: host ftruncate and reclaim cached pages beyond the new size
 // (Tab.1; used by the mat-vec output).
 __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
@@ -2098,7 +2350,7 @@ __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
   __syncthreads();
   if (tid == 0) {
     FileSnap s;
-    if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_GWRONCE)) {
+    if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_WRITABLE)) {
       sc.ret = -EBADF;
     } else {
       sc.fs = s;

@@ -29,6 +29,10 @@ extern "C" {
 /* ---- open flags ------------------------------------------ */
 #define GFS_O_RDONLY 0u
 #define GFS_O_GWRONCE 1u       /* write-once, pages never fetched, pristine = zeros */
+#define GFS_O_RDWR 2u          /* read-write with diff-and-merge write-back (NEXT-4):
+                                  pages fetched from the host, a pristine copy kept per dirty page */
+#define GFS_O_WRITABLE (GFS_O_GWRONCE | GFS_O_RDWR)
+#define GFS_PROT_WRITE 2u      /* gmmap prot: the mapping will be written (O_RDWR files) */
 #define GFS_O_PREFETCH 0x100u  /* gopen hint: fetch page 0 with the OPEN reply */
 
 /* ---- config flags ------------------------------------------------------ */
@@ -52,6 +56,7 @@ extern "C" {
 #define GFS_ST_ERROR (1u << 26)
 #define GFS_TAG_NONE 0xFFFFFFFFFFFFFFFFull /* tag = (uid << 32) | page index */
 #define GFS_DIRTY_NONE 0xFFFFFFFFu
+#define GFS_PRISTINE_PENDING 0xFFFFFFFFu
 
 /* ---- file table entry states (high byte of `sr`; low 24 bits = refcount) */
 #define GFS_FS_FREE 0u
@@ -91,6 +96,8 @@ typedef struct gfs_file {
 #define GFS_OP_TRUNC 5u    /* ftruncate(hfid, arg) */
 
 #define GFS_WF_FULL 1u     /* WRITE: every byte of [off,off+len) was written (no merge) */
+#define GFS_WF_DIFF 2u     /* WRITE (O_RDWR): write only the bytes where staging slot `stage` (working
+                              copy) differs from staging slot `arg` (pristine copy) */
 
 typedef struct gfs_rpc_req { /* one 64-byte ring slot in pinned host memory */
   uint32_t op;
@@ -188,6 +195,7 @@ typedef struct gfs_ctx {
   uint32_t* f_written;
   uint32_t* f_stamp;
   uint32_t* f_hv;     /* bytes [0, hv) equal the host file at the entry's version (peer fill) */
+  uint32_t* f_pristine; /* O_RDWR dirty page: pristine frame + 1 (0 none, GFS_PRISTINE_PENDING being made) */
   uint32_t* fresh_next;
   uint32_t* hand;
   /* radix node pool: 64-bit entries (interior: child node id; leaf: gen << 32 | frame + 1) */

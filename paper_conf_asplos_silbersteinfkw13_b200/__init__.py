@@ -25,6 +25,8 @@ HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", 
 
 O_RDONLY = 0
 O_GWRONCE = 1
+O_RDWR = 2
+PROT_WRITE = 2
 F_LOCKED_TRAVERSAL = 1
 F_NO_DMA_COMPLETION = 2
 DAEMON_SPAWN = 0
@@ -89,7 +91,8 @@ def lib():
             "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_randread_warp": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
-            "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32], I),
+            "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32, I], I),
+            "gfs_run_mmap_write": ([P, P, CS, U32, P, P, P, P, P, U32, U32, I], I),
             "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
             "gfs_run_seqwrite": ([P, P, CS, U64, U64, P, P, P, U32, U32, U32], I),
             "gfs_grep_work_bytes": ([ctypes.POINTER(gfs_grep_params)], U64),
@@ -204,9 +207,14 @@ def gfs_run_seqwrite(h, stream, path, total, chunk, d_src, d_err, d_tmp, grid, b
                                       sync_grid), "gfs_run_seqwrite")
 
 
-def gfs_run_gwrite(h, stream, path, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid, block):
+def gfs_run_gwrite(h, stream, path, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid, block, flags=1):
     return _ck(lib().gfs_run_gwrite(h, stream, _b(path), ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid,
-                                    block), "gfs_run_gwrite")
+                                    block, flags), "gfs_run_gwrite")
+
+
+def gfs_run_mmap_write(h, stream, path, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid, block, do_msync):
+    return _ck(lib().gfs_run_mmap_write(h, stream, _b(path), ncalls, d_off, d_len, d_srcoff, d_src, d_ret, grid,
+                                        block, do_msync), "gfs_run_mmap_write")
 
 
 def gfs_run_fileop(h, stream, path, flags, op, arg, d_ret):

@@ -89,7 +89,7 @@ class GpuFS:
         return torch.as_tensor(np.ascontiguousarray(a), device=f"cuda:{self.device}", dtype=dtype)
 
     # gread / gmmap parity harness -------------------------------------------
-    def gread_calls(self, path, offs, lens, mode=0, grid=None, block=256, smem=0, stream=None):
+    def gread_calls(self, path, offs, lens, mode=0, grid=None, block=256, smem=0, stream=None, open_flags=0):
         """Issue gread (mode 0), gmmap (1), gread-to-shared (2), gread-to-shared co-aligned with the
         offset (3), warp-collective gread_warp to global (4) or to per-warp shared (5) calls;
         returns (ret, dst, dstoff)."""
@@ -109,7 +109,7 @@ class GpuFS:
         if mode in (2, 3, 5) and smem == 0:
             smem = int(lens.max()) if n else 16
             smem = (smem + 15) // 16 * 16
-        gfs_run_gread(self.h, sp, path, mode, n, d_off.data_ptr(), d_len.data_ptr(), d_dstoff.data_ptr(),
+        gfs_run_gread(self.h, sp, path, mode | (open_flags << 8), n, d_off.data_ptr(), d_len.data_ptr(), d_dstoff.data_ptr(),
                       d_dst.data_ptr(), d_ret.data_ptr(), grid, block, smem)
         s.synchronize()
         return d_ret[:n].cpu().numpy(), d_dst.cpu().numpy(), dstoff
@@ -175,7 +175,10 @@ class GpuFS:
         return int(v[0].astype(np.uint64)), int(v[1])
 
     # gwrite -----------------------------------------------------------------
-    def gwrite_calls(self, path, offs, lens, data: bytes, srcoff=None, grid=None, block=256, stream=None):
+    def gwrite_calls(self, path, offs, lens, data: bytes, srcoff=None, grid=None, block=256, stream=None,
+                     flags=1, mmap=False, msync=True):
+        """gwrite harness (flags: O_GWRONCE = 1 or O_RDWR = 2). mmap=True instead writes
+        through gmmap(GFS_PROT_WRITE) pointers of an O_RDWR file (+ gmsync if msync)."""
         torch = _torch()
         offs = np.asarray(offs, dtype=np.uint64)
         lens = np.asarray(lens, dtype=np.uint64)
@@ -189,8 +192,14 @@ class GpuFS:
         d_srcoff = self._dev(np.asarray(srcoff, np.uint64).view(np.int64))
         d_ret = torch.full((max(n, 1),), -999, dtype=torch.int64, device=f"cuda:{self.device}")
         s, sp = self._stream(stream)
-        gfs_run_gwrite(self.h, sp, path, n, d_off.data_ptr(), d_len.data_ptr(), d_srcoff.data_ptr(),
-                       d_src.data_ptr(), d_ret.data_ptr(), grid or max(1, min(n, 296)), block)
+        if mmap:
+            from . import gfs_run_mmap_write
+            gfs_run_mmap_write(self.h, sp, path, n, d_off.data_ptr(), d_len.data_ptr(), d_srcoff.data_ptr(),
+                               d_src.data_ptr(), d_ret.data_ptr(), grid or max(1, min(n, 296)), block,
+                               1 if msync else 0)
+        else:
+            gfs_run_gwrite(self.h, sp, path, n, d_off.data_ptr(), d_len.data_ptr(), d_srcoff.data_ptr(),
+                           d_src.data_ptr(), d_ret.data_ptr(), grid or max(1, min(n, 296)), block, flags)
         s.synchronize()
         return d_ret[:n].cpu().numpy()
 
@@ -298,8 +307,8 @@ class GpuFS:
     def unpin(self, fd) -> int:
         return self.fileop("", "unpin", arg=fd)
 
-    def gfsync(self, path):
-        return self.fileop(path, "fsync", flags=1)
+    def gfsync(self, path, flags=1):
+        return self.fileop(path, "fsync", flags=flags)
 
     def gftruncate(self, path, size):
         return self.fileop(path, "ftruncate", flags=1, arg=size)

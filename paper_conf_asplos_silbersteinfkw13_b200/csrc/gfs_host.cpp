@@ -404,7 +404,7 @@ int w_fd(gfs_handle* h, Worker& w, uint32_t id) {
     ::close(it->second.fd);  // the hfid was recycled for another file
     w.fds.erase(it);
   }
-  const int fd = w_open_path(w, m.path, (m.mode & GFS_O_GWRONCE) ? O_RDWR : O_RDONLY);
+  const int fd = w_open_path(w, m.path, (m.mode & GFS_O_WRITABLE) ? O_RDWR : O_RDONLY);
   if (fd < 0) return -errno;
   struct stat st;
   if (fstat(fd, &st) != 0 || (uint64_t)st.st_dev != m.dev || (uint64_t)st.st_ino != m.ino) {
@@ -432,7 +432,7 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
   };
   gfs_rpc_resp* rs = h->resp_h + slot;
   std::string path(h->paths_h + (size_t)slot * GFS_MAX_PATH, q.path_len < GFS_MAX_PATH ? q.path_len : 0);
-  const bool gw = (q.flags & GFS_O_GWRONCE) != 0;
+  const bool gw = (q.flags & GFS_O_WRITABLE) != 0;
   int fd = w_open_path(w, path, gw ? (O_RDWR | O_CREAT) : O_RDONLY);
   if (fd < 0) {
     rs->status = -errno;
@@ -465,13 +465,13 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
     const uint32_t old = (uint32_t)(q.arg - 1);
     HostFile of;
     if (hfid_meta(h, old, &of) && of.dev == (uint64_t)st.st_dev && of.ino == (uint64_t)st.st_ino &&
-        (of.mode & GFS_O_GWRONCE) >= (q.flags & GFS_O_GWRONCE)) {
+        (!gw || (of.mode & GFS_O_WRITABLE))) {
       hfid = old;
       reused = true;
       // cache this fd only if it was opened as the hfid will be used: a
       // read-only re-open of a write-once hfid must not leave an O_RDONLY fd
       // where a later WRITE (pwrite) of the same hfid would find it
-      if (!(of.mode & GFS_O_GWRONCE) || gw) w_cache(w, hfid, fd, of.gen);
+      if (!(of.mode & GFS_O_WRITABLE) || gw) w_cache(w, hfid, fd, of.gen);
       else ::close(fd);
     } else {
       free_hfid(h, old);
@@ -513,7 +513,7 @@ const uint8_t* hfid_map(gfs_handle* h, Worker& w, uint32_t id, uint64_t* map_len
       *map_len = f.map_len;
       return f.map;
     }
-    if (f.map_tried || (f.mode & GFS_O_GWRONCE) || f.size < kMapMinBytes || h->nmapped >= kMapMaxFiles)
+    if (f.map_tried || (f.mode & GFS_O_WRITABLE) || f.size < kMapMinBytes || h->nmapped >= kMapMaxFiles)
       return nullptr;
     f.map_tried = true;  // one worker maps it; the others pread meanwhile
     size = f.size;
@@ -625,7 +625,11 @@ uint8_t* hfid_wmap(gfs_handle* h, Worker& w, uint32_t id, int fd, uint64_t end) 
     std::lock_guard<std::mutex> gg(h->grow_mu);
     struct stat st;
     if (fstat(fd, &st) != 0) return nullptr;
-    if ((uint64_t)st.st_size < end && ftruncate(fd, (off_t)end) != 0) return nullptr;
+    // fallocate only ever extends the size. ftruncate(end) here raced with a
+    // concurrent pwrite() (another worker, or the fallback path) that had just
+    // extended the file past `end`: it cut that write off (lost pages read
+    // back as zeros, ~5% of first-iteration C5 runs)
+    if ((uint64_t)st.st_size < end && fallocate(fd, 0, 0, (off_t)end) != 0) return nullptr;
     const uint64_t now = (uint64_t)st.st_size > end ? (uint64_t)st.st_size : end;
     std::lock_guard<std::mutex> g(h->fd_mu);
     HostFile& f = h->files[id];
@@ -638,12 +642,54 @@ uint8_t* hfid_wmap(gfs_handle* h, Worker& w, uint32_t id, int fd, uint64_t end) 
 int32_t do_write(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
   HostFile f;
   if (!hfid_meta(h, q.hfid, &f)) return -EBADF;
-  if (!(f.mode & GFS_O_GWRONCE)) return -EBADF;  // read-only files are never written back
+  if (!(f.mode & GFS_O_WRITABLE)) return -EBADF;  // read-only files are never written back
   const uint64_t in_page = q.file_off & (h->h.page_size - 1);
   if (in_page + q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
   const int fd = w_fd(h, w, q.hfid);
   if (fd < 0) return fd;
   uint8_t* buf = staging_slot(h, q.stage) + in_page;
+  if (q.flags & GFS_WF_DIFF) {
+    // O_RDWR diff-and-merge: write back exactly the bytes where
+    // the working copy differs from the pristine one, as runs, so bytes other
+    // writers changed in the same page are never reverted
+    if (!(f.mode & GFS_O_RDWR) || q.arg >= h->h.staging_slots) return -EINVAL;
+    const uint8_t* pri = staging_slot(h, (uint32_t)q.arg) + in_page;
+    {  // the write ends at file_off + len: the file is at least that long, even if
+       // its last bytes equal the pristine copy (zeros past the old EOF).
+       // fallocate only ever grows the size (concurrent writers never shrink it).
+      const uint64_t end = q.file_off + q.len;
+      struct stat stt;
+      if (fstat(fd, &stt) == 0 && (uint64_t)stt.st_size < end &&
+          fallocate(fd, 0, (off_t)q.file_off, (off_t)q.len) != 0) {
+        std::lock_guard<std::mutex> g(h->grow_mu);
+        if (fstat(fd, &stt) == 0 && (uint64_t)stt.st_size < end && ftruncate(fd, (off_t)end) != 0) return -errno;
+      }
+    }
+    uint8_t* wm = nullptr;
+    bool wm_ok = true;
+    uint64_t i = 0, runs = 0;
+    while (i < q.len) {
+      while (i < q.len && buf[i] == pri[i]) ++i;  // (a memcmp-by-words scan would be faster; pages are small)
+      if (i >= q.len) break;
+      uint64_t j = i;
+      while (j < q.len && buf[j] != pri[j]) ++j;
+      if (!wm && wm_ok) {
+        wm = hfid_wmap(h, w, q.hfid, fd, q.file_off + q.len);
+        wm_ok = wm != nullptr;
+      }
+      if (!(wm && map_store(wm, buf + i, q.file_off + i, j - i))) {
+        const int64_t r = pwrite_full(fd, buf + i, j - i, q.file_off + i);
+        if (r < 0) return (int32_t)r;
+      }
+      ++runs;
+      h->hs[HS_BYTES_D2H] += j - i;
+      i = j;
+    }
+    h->resp_h[slot].version = h->vt.bump(f.dev, f.ino);
+    h->hs[HS_WRITE]++;
+    h->hs[HS_MERGES]++;
+    return (int32_t)q.len;
+  }
   if (!(q.flags & GFS_WF_FULL)) {
     // Not every byte of the range was written: diff against zeros.
     w.merge.assign(q.len, 0);
@@ -771,7 +817,7 @@ void free_all(gfs_handle* h) {
   h->ipc_open.clear();
   if (h->own_pool) F(h->h.pool);
   F(h->h.f_state); F(h->h.f_tag); F(h->h.f_file); F(h->h.f_valid); F(h->h.f_lo); F(h->h.f_hi);
-  F(h->h.f_written); F(h->h.f_stamp); F(h->h.f_hv); F((void*)h->h.peers); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
+  F(h->h.f_written); F(h->h.f_stamp); F(h->h.f_hv); F(h->h.f_pristine); F((void*)h->h.peers); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
   F(h->h.node_free); F(h->h.node_free_top); F(h->h.node_lock); F(h->h.files); F(h->h.paths); F(h->h.uid_next);
   F(h->h.ack); F(h->h.ring_tail); F(h->h.ctr); F(h->h.staging_bits); F(h->d);
   if (h->ring_h) cudaFreeHost(h->ring_h);
@@ -869,6 +915,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMalloc((void**)&c.f_written, nframes * 4));
   CK(cudaMalloc((void**)&c.f_stamp, nframes * 4));
   CK(cudaMalloc((void**)&c.f_hv, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_pristine, nframes * 4));
   CK(cudaMalloc((void**)&c.fresh_next, 4));
   CK(cudaMalloc((void**)&c.hand, 4));
   c.max_nodes = max_nodes;

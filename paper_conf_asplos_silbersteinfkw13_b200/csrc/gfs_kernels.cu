@@ -34,6 +34,7 @@ __global__ void k_init_metadata(gfs_ctx c) {
     c.f_written[i] = 0;
     c.f_stamp[i] = 0;
     c.f_hv[i] = 0;
+    c.f_pristine[i] = 0;
   }
   if (blockIdx.x == 0 && threadIdx.x == 0) {
     *c.fresh_next = 0;
@@ -93,7 +94,8 @@ __global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint
                               uint32_t smem_bytes) {
   extern __shared__ __align__(16) uint8_t smem[];
   const int tid = threadIdx.x;
-  const int fd = gopen(c, path, GFS_O_RDONLY);
+  const int fd = gopen(c, path, mode >> 8);  // open flags ride in the high bits (O_RDONLY or O_RDWR)
+  mode &= 0xFF;
   for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
     int64_t r;
     if (fd < 0) {
@@ -311,10 +313,43 @@ __global__ void __launch_bounds__(256) k_randread_warp(const gfs_ctx* c, const c
 }
 
 __global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
-                               const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret) {
-  const int fd = gopen(c, path, GFS_O_GWRONCE);
+                               const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret,
+                               int flags) {
+  const int fd = gopen(c, path, flags);
   for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
     int64_t r = fd < 0 ? fd : gwrite(c, fd, off[i], len[i], src + srcoff[i]);
+    if (threadIdx.x == 0) ret[i] = r;
+  }
+  if (fd >= 0) gclose(c, fd);
+}
+
+// Writable-mapping harness (O_RDWR, Tab.1 gmsync): block i maps
+// [off[i], off[i] + len[i]) with GFS_PROT_WRITE, stores src bytes through the
+// pointer, optionally gmsync()s the page, and gmunmap()s. ret[i] = bytes
+// mapped (the prefix) or -errno.
+__global__ void k_mmap_write(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
+                             const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret,
+                             int do_msync) {
+  const int fd = gopen(c, path, GFS_O_RDWR);
+  for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
+    int64_t r = fd;
+    if (fd >= 0) {
+      uint64_t m = 0;
+      uint8_t* p = (uint8_t*)gmmap(c, nullptr, len[i], GFS_PROT_WRITE, 0, fd, off[i], &m);
+      if (!p) {
+        r = m ? -EIO : (int64_t)-EBADF;
+      } else {
+        for (uint64_t k = threadIdx.x; k < m; k += blockDim.x) p[k] = src[srcoff[i] + k];
+        __threadfence();
+        __syncthreads();
+        r = (int64_t)m;
+        if (do_msync) {
+          const int e = gmsync(c, p, m, 0);
+          if (e < 0) r = e;
+        }
+        gmunmap(c, p, m);
+      }
+    }
     if (threadIdx.x == 0) ret[i] = r;
   }
   if (fd >= 0) gclose(c, fd);
@@ -434,12 +469,14 @@ extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s) {
 GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint32_t ncalls,
                           const uint64_t* d_off, const uint64_t* d_len, const uint64_t* d_dstoff, uint8_t* d_dst,
                           int64_t* d_ret, uint32_t grid, uint32_t block, uint32_t smem_bytes) {
-  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || mode > 5) return -EINVAL;
-  if (mode >= 4 && ((block & 31) || block > 32 * GFS_WARP_API_MAX_WARPS)) return -EINVAL;
+  if (!h || grid == 0 || block == 0 || block > 1024 || mode < 0 || (mode & 0xFF) > 5) return -EINVAL;
+  if ((mode >> 8) != (int)GFS_O_RDONLY && (mode >> 8) != (int)GFS_O_RDWR) return -EINVAL;
+  if ((mode & 0xFF) >= 4 && (mode >> 8)) return -EINVAL;  // warp harness: read-only opens
+  if ((mode & 0xFF) >= 4 && ((block & 31) || block > 32 * GFS_WARP_API_MAX_WARPS)) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
   const char* dp = stage_path(path, s);
   if (!dp) return -ENAMETOOLONG;
-  if (mode >= 4) {
+  if (mode >= 4 && mode <= 5) {
     const uint32_t dyn = mode == 5 ? smem_bytes * (block / 32) : 0;
     if (dyn > 200 * 1024) return -EINVAL;
     if (dyn > 48 * 1024)
@@ -448,9 +485,9 @@ GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mod
                                                 d_ret, smem_bytes);
     return launch_err(cudaGetLastError());
   }
-  if (mode >= 2 && smem_bytes > 48 * 1024)
+  if ((mode & 0xFF) >= 2 && smem_bytes > 48 * 1024)
     cudaFuncSetAttribute(k_gread_calls, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem_bytes);
-  k_gread_calls<<<grid, block, mode >= 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,
+  k_gread_calls<<<grid, block, (mode & 0xFF) >= 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,
                                                                 d_dstoff, d_dst, d_ret, smem_bytes);
   return launch_err(cudaGetLastError());
 }
@@ -499,12 +536,24 @@ GFS_API int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path,
 
 GFS_API int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32_t ncalls, const uint64_t* d_off,
                            const uint64_t* d_len, const uint64_t* d_srcoff, const uint8_t* d_src, int64_t* d_ret,
-                           uint32_t grid, uint32_t block) {
+                           uint32_t grid, uint32_t block, int flags) {
+  if (!h || grid == 0 || block == 0 || block > 1024) return -EINVAL;
+  if (flags != (int)GFS_O_GWRONCE && flags != (int)GFS_O_RDWR) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  const char* dp = stage_path(path, s);
+  if (!dp) return -ENAMETOOLONG;
+  k_gwrite_calls<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, flags);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_mmap_write(gfs_handle* h, void* stream, const char* path, uint32_t ncalls, const uint64_t* d_off,
+                               const uint64_t* d_len, const uint64_t* d_srcoff, const uint8_t* d_src, int64_t* d_ret,
+                               uint32_t grid, uint32_t block, int do_msync) {
   if (!h || grid == 0 || block == 0 || block > 1024) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
   const char* dp = stage_path(path, s);
   if (!dp) return -ENAMETOOLONG;
-  k_gwrite_calls<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret);
+  k_mmap_write<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, do_msync);
   return launch_err(cudaGetLastError());
 }
 
