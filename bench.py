@@ -676,7 +676,64 @@ def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
     })
     if local_peer:
         res["read_peer_same_gpu"] = local_peer
+    if ws == 1 and not args.no_rdwr:
+        res["rdwr_shared_pages"] = rdwr_phase(args, torch, g, dev)
     return res
+
+
+def rdwr_phase(args, torch, g, dev):
+    """NEXT-4: two caches (stand-ins for two GPUs) open one existing
+    file O_RDWR and write interleaved 64 KiB blocks of every 2 MiB page (false
+    sharing), then gfsync: each write-back sends only the bytes that differ from
+    the page's pristine copy, so both halves survive. Parity: the host file
+    equals the original with both writers' blocks laid over it."""
+    P, blk = 2 << 20, 64 << 10
+    size = args.rdwr_mib << 20
+    root = "/dev/shm/gfs_bench_rdwr"
+    os.makedirs(root, exist_ok=True)
+    path = f"{root}/shared.bin"
+    orig = np.random.default_rng(900).integers(0, 256, size=size, dtype=np.uint8)
+    orig.tofile(path)
+    offs = np.arange(0, size, blk, dtype=np.uint64)
+    new = np.random.default_rng(901).integers(0, 256, size=size, dtype=np.uint8)
+    times = {"gwrite": [], "gfsync": []}
+    caches = [g.GpuFS(cache_bytes=2 * size + (256 << 20), page_size=P, device=torch.cuda.current_device(),
+                      daemon_threads=args.daemon_threads, max_batch=8, timeout_ms=args.timeout_ms)
+              for _ in range(2)]
+    try:
+        fds = [c.pin(path, flags=g.O_RDWR) for c in caches]
+        for k, c in enumerate(caches):
+            mine = offs[k::2]
+            data = np.concatenate([new[int(o):int(o) + blk] for o in mine]).tobytes()
+            e = [torch.cuda.Event(enable_timing=True) for _ in range(4)]
+            torch.cuda.synchronize()
+            e[0].record()
+            ret = c.gwrite_calls(path, mine, np.full(len(mine), blk, np.uint64), data, grid=296, flags=g.O_RDWR)
+            e[1].record()
+            assert (ret == blk).all(), ret[:4]
+            e[2].record()
+            r = c.gfsync(path, flags=g.O_RDWR, grid=64)
+            e[3].record()
+            torch.cuda.synchronize()
+            assert r == 0, r
+            times["gwrite"].append(e[0].elapsed_time(e[1]))
+            times["gfsync"].append(e[2].elapsed_time(e[3]))
+        for c, fd in zip(caches, fds):
+            c.unpin(fd)
+        st = [c.stats() for c in caches]
+    finally:
+        for c in caches:
+            c.close()
+    host = np.fromfile(path, dtype=np.uint8)
+    ok = host.size == size and np.array_equal(host, new)  # every block came from one of the two writers
+    half = size / 2
+    return {"workload": f"two caches, one {args.rdwr_mib} MiB file O_RDWR, 2 MiB pages, interleaved 64 KiB blocks "
+                        f"(every page written by both), gwrite then gfsync per cache; one GPU",
+            "gwrite_GBps": round(half / (float(np.mean(times["gwrite"])) * 1e-3) / 1e9, 3),
+            "gfsync_GBps": round(half / (float(np.mean(times["gfsync"])) * 1e-3) / 1e9, 3),
+            "parity": bool(ok), "writebacks": [x["writeback"] for x in st], "misses": [x["miss"] for x in st],
+            "note": "gwrite includes the page fetches (O_RDWR reads pages) and pristine copies; gfsync moves "
+                    "working + pristine ranges over PCIe and the host writes only changed bytes"}
 
 
 def c5_local_peer(args, torch, g, fs, path, size, P, grid, dev, stream, scratch, out):
@@ -752,6 +809,8 @@ def main():
     ap.add_argument("--grep-cache-gib", type=int, default=4)
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--no-peers", action="store_true", help="C5 without peer-cache fill (NEXT-1)")
+    ap.add_argument("--no-rdwr", action="store_true", help="skip the O_RDWR shared-page phase (NEXT-4)")
+    ap.add_argument("--rdwr-mib", type=int, default=256)
     args = ap.parse_args()
     if args.impl == "reference":
         run_reference(args)

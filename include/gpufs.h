@@ -191,7 +191,9 @@ int gfs_run_mmap_write(gfs_handle* h, void* stream, const char* path, uint32_t n
 
 /* One-block file operations: op 0 = gfsync, 1 = gftruncate(arg), 2 = gfstat_size,
  * 3 = gopen+gclose only, 4 = pin (gopen without gclose: the file stays open
- * across launches, *d_ret = fd), 5 = unpin (gclose(fd = arg)).
+ * across launches, *d_ret = fd), 5 = unpin (gclose(fd = arg)), 6 = gfsync from `arg`
+ * blocks at once (they split the dirty pages by claim) followed by a strict
+ * one-block pass; *d_ret = 0 or the most negative error.
  * flags = open flags. *d_ret = result. */
 /* C5 write side: pin `path` open O_GWRONCE (one
  * reference held for the duration), then `grid` blocks gwrite() [0, total)

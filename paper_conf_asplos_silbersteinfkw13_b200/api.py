@@ -206,7 +206,7 @@ class GpuFS:
     def fileop(self, path, op, flags=0, arg=0, stream=None) -> int:
         """op: 'fsync' | 'ftruncate' | 'fstat' | 'openclose'."""
         torch = _torch()
-        code = {"fsync": 0, "ftruncate": 1, "fstat": 2, "openclose": 3, "pin": 4, "unpin": 5}[op]
+        code = {"fsync": 0, "ftruncate": 1, "fstat": 2, "openclose": 3, "pin": 4, "unpin": 5, "fsync_grid": 6}[op]
         d_ret = torch.full((1,), -999, dtype=torch.int64, device=f"cuda:{self.device}")
         s, sp = self._stream(stream)
         gfs_run_fileop(self.h, sp, path, flags, code, arg, d_ret.data_ptr())
@@ -307,7 +307,10 @@ class GpuFS:
     def unpin(self, fd) -> int:
         return self.fileop("", "unpin", arg=fd)
 
-    def gfsync(self, path, flags=1):
+    def gfsync(self, path, flags=1, grid=1):
+        """gfsync(path) from one block, or from `grid` blocks at once (+ a strict pass)."""
+        if grid > 1:
+            return self.fileop(path, "fsync_grid", flags=flags, arg=grid)
         return self.fileop(path, "fsync", flags=flags)
 
     def gftruncate(self, path, size):

@@ -400,6 +400,18 @@ __global__ void k_unpin(const gfs_ctx* c, const int64_t* pinned_fd, int64_t* err
 }
 
 __global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, uint64_t arg, int64_t* ret) {
+  if (op == 6) {  // gfsync from every block of the grid (the pages split by claim), then a strict pass
+    const int fd = gopen(c, path, flags);
+    int r = fd;
+    if (fd >= 0) {
+      r = gfsync(c, fd);
+      if (arg == 0 && r == -EBUSY) r = 0;  // a page another block of this grid was syncing
+      const int cr = gclose(c, fd);
+      if (r >= 0 && cr < 0) r = cr;
+    }
+    if (threadIdx.x == 0 && r < 0) atomicMin((long long*)ret, (long long)r);
+    return;
+  }
   if (op == 5) {  // unpin: drop a reference taken by op 4
     const int64_t r = gclose(c, (int)arg);
     if (threadIdx.x == 0) *ret = r;
@@ -582,6 +594,13 @@ GFS_API int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int fl
   cudaStream_t s = (cudaStream_t)stream;
   const char* dp = stage_path(path, s);
   if (!dp) return -ENAMETOOLONG;
+  if (op == 6) {  // parallel gfsync: arg = grid; *d_ret = 0 or the most negative error
+    if (arg == 0 || arg > 65535) return -EINVAL;
+    cudaMemsetAsync(d_ret, 0, 8, s);
+    k_fileop<<<(uint32_t)arg, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, 6, 0, d_ret);
+    k_fileop<<<1, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, 6, 1, d_ret);  // strict: every page clean now
+    return launch_err(cudaGetLastError());
+  }
   k_fileop<<<1, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, op, arg, d_ret);
   return launch_err(cudaGetLastError());
 }

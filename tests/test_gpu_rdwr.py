@@ -98,7 +98,7 @@ def test_rdwr_two_writers_share_pages(g, shmdir):
             ret = fs.gwrite_calls(path, [o for o, _ in ws], [len(b) for _, b in ws], b"".join(b for _, b in ws),
                                   grid=8, flags=RDWR)
             assert (ret == 40).all()
-        assert A.gfsync(path, flags=RDWR) == 0
+        assert A.gfsync(path, flags=RDWR, grid=8) == 0  # many blocks share the write-back
         assert B.gfsync(path, flags=RDWR) == 0
         A.unpin(fa)
         B.unpin(fb)
