@@ -747,7 +747,7 @@ __device__ __forceinline__ void pristine_free(const gfs_ctx* c, uint32_t f) {
 
 // Write back a frame's dirty range from one thread (the caller owns the frame:
 // EVICTING, ref 0): copy it into a staging slot over PCIe, then WRITE RPC.
-__device__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
+__device__ __noinline__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
   const uint32_t lo = ld_rlx(&c->f_lo[f]);
   if (lo == GFS_DIRTY_NONE) return 0;
   const uint32_t hi = ld_rlx(&c->f_hi[f]);
@@ -814,7 +814,7 @@ __device__ __forceinline__ uint32_t frame_tier(const gfs_ctx* c, uint32_t f, uin
 // writing back a dirty victim first. Runs in the calling thread.
 // Returns the frame in state FILLING|1 with its tag set (and its new
 // generation in *gen), or -ENOMEM.
-__device__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx, uint32_t* gen) {
+__device__ __noinline__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx, uint32_t* gen) {
   const uint32_t N = c->nframes;
   if (ld_rlx(c->fresh_next) < N) {
     const uint32_t f = atomicAdd(c->fresh_next, 1u);
@@ -961,7 +961,7 @@ __device__ __forceinline__ bool peek_busy(const gfs_ctx* c, const FileSnap& fs, 
 // the peer's eviction skips referenced frames. Result code (k << 27) | f, or
 // -1 when no peer has a usable copy.
 constexpr uint32_t kPeerFrameBits = 27;
-__device__ int peer_take(const gfs_ctx* c, const FileSnap& fs, uint64_t page, uint32_t nb) {
+__device__ __noinline__ int peer_take(const gfs_ctx* c, const FileSnap& fs, uint64_t page, uint32_t nb) {
   const gfs_file* me = c->files + fs.fdx;
   const uint64_t h = ld_rlx64(&me->path_hash);
   const uint32_t n = ld_rlx(&me->path_len);
@@ -1046,7 +1046,7 @@ struct Lk {
 // page has been pread by the host into staging slot `stage` (READ RPC,
 // P:L570-576); for O_GWRONCE files nothing is fetched. The
 // caller's block fills the frame and clears FILLING.
-__device__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
+__device__ __noinline__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint64_t page) {
   Lk out{kBusy, -1, 0, 0};
   const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)page;
   uint32_t* lockp = &c->files[fs.fdx].lock;
@@ -1287,7 +1287,7 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
 // another block is making is waited for (that block only copies a frame it
 // holds: it never waits on us). Returns 0 or -errno (then no claim is left).
 template <class G = BlockGroup>
-__device__ int ensure_pristine(const gfs_ctx* c, Scratch& sc, uint32_t fdx, uint32_t cnt) {
+__device__ __noinline__ int ensure_pristine(const gfs_ctx* c, Scratch& sc, uint32_t fdx, uint32_t cnt) {
   const int tid = G::tid(), nthr = G::nthr();
   if (tid == 0) sc.err = 0;
   if (tid < (int)cnt) {
@@ -1786,6 +1786,78 @@ __device__ inline int64_t gfstat_size_t(const gfs_ctx* c, int fd) {
   return sc.ret;
 }
 
+// gread past its first barrier when the call is not a one-page shared-memory
+// hit: the page batches (misses, multi-page spans, global destinations). Kept
+// out of line so the hit path's registers are not shaped by this code.
+template <class G>
+__device__ __noinline__ int64_t gread_batches(const gfs_ctx* c, int64_t n, uint64_t off, void* dst) {
+  using namespace detail;
+  Scratch& sc = G::sc();
+  const int tid = G::tid(), nthr = G::nthr();
+  const uint32_t shift = c->page_shift;
+  const uint64_t P = c->page_size;
+  const uint32_t B = c->max_batch < (uint32_t)nthr ? c->max_batch : (uint32_t)nthr;
+  const FileSnap fs = sc.fs;
+  const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
+  // TMA path: shared-memory destination co-aligned with the file offset
+  // ((dst - off) % 16 == 0, so frame and destination agree mod 16): aligned
+  // middles by TMA, the call's head and tail bytes by warp 0.
+  const bool tma = __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0;
+  for (uint64_t pb = p0; pb <= p1; pb += B) {
+    const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
+    const int err = acquire_batch<G>(c, sc, fs, pb, cnt, pb == p0);
+    if (err) return err;
+    const uint64_t bs = pb == p0 ? (off & (P - 1)) : 0;
+    const uint64_t be = pb + cnt - 1 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+    const uint64_t batch_bytes = ((uint64_t)cnt << shift) - bs - (P - be);
+    if (tma && batch_bytes < (1u << 20)) {  // mbarrier tx-count limit
+      const uint32_t ph = sc.mbar_phase;
+      if (tid == 0) {
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
+        uint32_t tx = 0;
+        for (uint32_t i = 0; i < cnt; ++i) {  // interior pages are whole and aligned: only the
+          const uint64_t p = pb + i;          // call's first and last pages have edges
+          const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+          const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+          tx += span_mid(frame_ptr(c, (uint32_t)sc.frame[i]) + s, (uint32_t)(e - s));
+        }
+        mbar_expect_tx(&sc.mbar, tx);
+        for (uint32_t i = 0; i < cnt; ++i) {
+          const uint64_t p = pb + i;
+          const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+          const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+          tma_span((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+                   (uint32_t)(e - s), &sc.mbar);
+        }
+      }
+      if (tid < 32) {
+        if (pb == p0) {
+          const uint64_t s = off & (P - 1), e = p0 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+          copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + s, (uint32_t)(e - s), tid);
+        }
+        if (pb + cnt - 1 == p1 && p1 != p0) {
+          const uint64_t e = ((off + (uint64_t)n - 1) & (P - 1)) + 1;
+          copy_edges((uint8_t*)dst + ((p1 << shift) - off), frame_ptr(c, (uint32_t)sc.frame[cnt - 1]), (uint32_t)e, tid);
+        }
+      }
+      mbar_wait(&sc.mbar, ph);
+      G::sync();
+      if (tid == 0) sc.mbar_phase = ph ^ 1u;
+    } else {
+      for (uint32_t i = 0; i < cnt; ++i) {
+        const uint64_t p = pb + i;
+        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
+        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
+        block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
+                              e - s, tid, nthr);
+      }
+      G::sync();
+    }
+    if (tid < (int)cnt) frame_release(c, (uint32_t)sc.frame[tid]);
+  }
+  return n;
+}
+
 // gread: pread semantics; returns min(len, S-off) bytes, 0 at/after EOF.
 template <class G>
 __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
@@ -1865,65 +1937,7 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
     }
     return n;
   }
-  const FileSnap fs = sc.fs;
-  const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)n - 1) >> shift;
-  // TMA path: shared-memory destination co-aligned with the file offset
-  // ((dst - off) % 16 == 0, so frame and destination agree mod 16): aligned
-  // middles by TMA, the call's head and tail bytes by warp 0.
-  const bool tma = __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0;
-  for (uint64_t pb = p0; pb <= p1; pb += B) {
-    const uint32_t cnt = (uint32_t)((p1 - pb + 1) < B ? (p1 - pb + 1) : B);
-    const int err = acquire_batch<G>(c, sc, fs, pb, cnt, pb == p0);
-    if (err) return err;
-    const uint64_t bs = pb == p0 ? (off & (P - 1)) : 0;
-    const uint64_t be = pb + cnt - 1 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-    const uint64_t batch_bytes = ((uint64_t)cnt << shift) - bs - (P - be);
-    if (tma && batch_bytes < (1u << 20)) {  // mbarrier tx-count limit
-      const uint32_t ph = sc.mbar_phase;
-      if (tid == 0) {
-        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
-        uint32_t tx = 0;
-        for (uint32_t i = 0; i < cnt; ++i) {  // interior pages are whole and aligned: only the
-          const uint64_t p = pb + i;          // call's first and last pages have edges
-          const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
-          const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-          tx += span_mid(frame_ptr(c, (uint32_t)sc.frame[i]) + s, (uint32_t)(e - s));
-        }
-        mbar_expect_tx(&sc.mbar, tx);
-        for (uint32_t i = 0; i < cnt; ++i) {
-          const uint64_t p = pb + i;
-          const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
-          const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-          tma_span((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
-                   (uint32_t)(e - s), &sc.mbar);
-        }
-      }
-      if (tid < 32) {
-        if (pb == p0) {
-          const uint64_t s = off & (P - 1), e = p0 == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-          copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + s, (uint32_t)(e - s), tid);
-        }
-        if (pb + cnt - 1 == p1 && p1 != p0) {
-          const uint64_t e = ((off + (uint64_t)n - 1) & (P - 1)) + 1;
-          copy_edges((uint8_t*)dst + ((p1 << shift) - off), frame_ptr(c, (uint32_t)sc.frame[cnt - 1]), (uint32_t)e, tid);
-        }
-      }
-      mbar_wait(&sc.mbar, ph);
-      G::sync();
-      if (tid == 0) sc.mbar_phase = ph ^ 1u;
-    } else {
-      for (uint32_t i = 0; i < cnt; ++i) {
-        const uint64_t p = pb + i;
-        const uint64_t s = p == p0 ? (off & (P - 1)) : 0;
-        const uint64_t e = p == p1 ? ((off + (uint64_t)n - 1) & (P - 1)) + 1 : P;
-        block_copy_from_frame((uint8_t*)dst + ((p << shift) + s - off), frame_ptr(c, (uint32_t)sc.frame[i]) + s,
-                              e - s, tid, nthr);
-      }
-      G::sync();
-    }
-    if (tid < (int)cnt) frame_release(c, (uint32_t)sc.frame[tid]);
-  }
-  return n;
+  return gread_batches<G>(c, n, off, dst);
 }
 
 // Threadblock-collective calls (the prototype's granularity).

@@ -120,7 +120,9 @@ def test_peer_fill_under_peer_eviction(g, shmdir):
     size = 48 * P + 5
     path = gen.splitmix_file(os.path.join(shmdir, "ev.bin"), size, seed=13)
     with g.GpuFS(cache_bytes=12 * P, page_size=P, timeout_ms=30000, daemon_threads=2) as A, \
-            g.GpuFS(cache_bytes=8 * P, page_size=P, timeout_ms=30000, daemon_threads=2) as B:
+            g.GpuFS(cache_bytes=16 * P, page_size=P, timeout_ms=30000, daemon_threads=2) as B:
+        # B: 4 blocks hold up to 3 pages each (2P spans): 16 frames keep the
+        # deadlock guard's bound (frames >= blocks x pages held) with slack
         B.attach_peer(A.export())
         s, err = A.seqread(path, size - size % 8, P, grid=4)
         assert err == 0
