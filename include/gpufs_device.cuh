@@ -1279,6 +1279,36 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
   }
 }
 
+// O_RDWR write-back with the diff done on the GPU: for frame f
+// and its pristine copy pf, bytes [lo, hi) of the page (lo a multiple of 64)
+// go to staging slot `st` (working copy, at in-page offsets) and a bitmap to
+// slot `mst`: bit j of 64-bit word w <=> byte lo + 64w + j differs. The host
+// writes only those bytes (GFS_WF_MASK). PCIe carries 1 + 1/8 bytes per dirty
+// byte instead of 2 (working + pristine). Block-collective.
+__device__ __forceinline__ void diff_to_stage(const gfs_ctx* c, uint32_t f, uint32_t pf, uint32_t lo, uint32_t hi,
+                                              int st, int mst, int tid, int nthr) {
+  const uint8_t* w = frame_ptr(c, f) + lo;
+  const uint8_t* p = frame_ptr(c, pf) + lo;
+  uint8_t* out = stage_ptr(c, st) + lo;
+  uint64_t* mask = (uint64_t*)stage_ptr(c, mst);
+  const uint32_t nw = (hi - lo + 63) / 64;
+  for (uint32_t k = tid; k < nw; k += nthr) {
+    uint64_t m = 0;
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      const int4 a = __ldcg((const int4*)(w + 64 * k) + q), b = __ldcg((const int4*)(p + 64 * k) + q);
+      ((int4*)(out + 64 * k))[q] = a;
+      const uint32_t d[4] = {__vcmpne4(a.x, b.x), __vcmpne4(a.y, b.y), __vcmpne4(a.z, b.z), __vcmpne4(a.w, b.w)};
+#pragma unroll
+      for (int j = 0; j < 4; ++j)  // 0xFF/0x00 per byte -> 4 bits (as word_bits4 in the grep scan)
+        m |= (uint64_t)((((d[j] >> 7) & 0x01010101u) * 0x00204081u) >> 21 & 0xFu) << (16 * q + 4 * j);
+    }
+    const uint32_t end = lo + 64 * k + 64;
+    if (end > hi) m &= (hi - (lo + 64 * k) >= 64) ? ~0ull : ((1ull << (hi - (lo + 64 * k))) - 1ull);
+    mask[k] = m;
+  }
+}
+
 // O_RDWR: before the first local write to a page, preserve its
 // pristine copy. Block-collective over the held frames sc.frame[0, cnt): lane
 // i claims the pristine slot of page i (CAS 0 -> PENDING), allocates a frame
@@ -2114,11 +2144,13 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
       __syncthreads();
       for (uint32_t i = 0; i < cnt; ++i)
         if (sc.frame[i] >= 0) {
-          block_copy_from_frame(stage_ptr(c, sc.stage[i]) + sc.lo[i], frame_ptr(c, (uint32_t)sc.frame[i]) + sc.lo[i],
-                                sc.hi[i] - sc.lo[i], tid, nthr);
-          if (sc.nbytes[i])
-            block_copy_from_frame(stage_ptr(c, (int)sc.fill[i]) + sc.lo[i], frame_ptr(c, sc.nbytes[i] - 1) + sc.lo[i],
-                                  sc.hi[i] - sc.lo[i], tid, nthr);
+          if (sc.nbytes[i]) {  // O_RDWR: the GPU diffs; the host gets the working bytes + a changed-byte mask
+            diff_to_stage(c, (uint32_t)sc.frame[i], sc.nbytes[i] - 1, sc.lo[i] & ~63u, sc.hi[i], sc.stage[i],
+                          (int)sc.fill[i], tid, nthr);
+          } else {
+            block_copy_from_frame(stage_ptr(c, sc.stage[i]) + sc.lo[i],
+                                  frame_ptr(c, (uint32_t)sc.frame[i]) + sc.lo[i], sc.hi[i] - sc.lo[i], tid, nthr);
+          }
         }
       __threadfence_system();
       __syncthreads();
@@ -2127,9 +2159,10 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
         const uint32_t lo = sc.lo[tid], hi = sc.hi[tid];
         const uint32_t wr = ld_rlx(&c->f_written[f]);
         const bool diff = sc.nbytes[tid] != 0;
+        const uint32_t lo_w = diff ? (lo & ~63u) : lo;  // the mask covers whole 64-byte words
         gfs_rpc_resp rs;
-        const int32_t r = rpc_call(c, GFS_OP_WRITE, fs.hfid, ((pb + tid) << c->page_shift) + lo, sc.stage[tid],
-                                   hi - lo, diff ? GFS_WF_DIFF : (wr >= hi - lo ? GFS_WF_FULL : 0u),
+        const int32_t r = rpc_call(c, GFS_OP_WRITE, fs.hfid, ((pb + tid) << c->page_shift) + lo_w, sc.stage[tid],
+                                   hi - lo_w, diff ? GFS_WF_MASK : (wr >= hi - lo ? GFS_WF_FULL : 0u),
                                    diff ? (uint64_t)sc.fill[tid] : 0, nullptr, 0, &rs);
         stage_free(c, sc.stage[tid]);
         if (diff) stage_free(c, (int)sc.fill[tid]);

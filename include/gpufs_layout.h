@@ -98,6 +98,9 @@ typedef struct gfs_file {
 #define GFS_WF_FULL 1u     /* WRITE: every byte of [off,off+len) was written (no merge) */
 #define GFS_WF_DIFF 2u     /* WRITE (O_RDWR): write only the bytes where staging slot `stage` (working
                               copy) differs from staging slot `arg` (pristine copy) */
+#define GFS_WF_MASK 4u     /* WRITE (O_RDWR): staging slot `arg` holds a bitmap over [off, off+len)
+                              (64-bit words, bit j of word w = byte 64w + j; off is 64-aligned in the
+                              page): write only the marked bytes of slot `stage` */
 
 typedef struct gfs_rpc_req { /* one 64-byte ring slot in pinned host memory */
   uint32_t op;

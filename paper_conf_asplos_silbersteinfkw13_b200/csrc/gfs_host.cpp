@@ -648,12 +648,15 @@ int32_t do_write(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) 
   const int fd = w_fd(h, w, q.hfid);
   if (fd < 0) return fd;
   uint8_t* buf = staging_slot(h, q.stage) + in_page;
-  if (q.flags & GFS_WF_DIFF) {
+  if (q.flags & (GFS_WF_DIFF | GFS_WF_MASK)) {
     // O_RDWR diff-and-merge: write back exactly the bytes where
     // the working copy differs from the pristine one, as runs, so bytes other
     // writers changed in the same page are never reverted
     if (!(f.mode & GFS_O_RDWR) || q.arg >= h->h.staging_slots) return -EINVAL;
-    const uint8_t* pri = staging_slot(h, (uint32_t)q.arg) + in_page;
+    const bool bits = (q.flags & GFS_WF_MASK) != 0;  // GPU-made changed-byte mask instead of a pristine copy
+    const uint8_t* pri = staging_slot(h, (uint32_t)q.arg) + (bits ? 0 : in_page);
+    const uint64_t* mw = (const uint64_t*)staging_slot(h, (uint32_t)q.arg);
+    auto changed = [&](uint64_t i) { return bits ? ((mw[i >> 6] >> (i & 63)) & 1) != 0 : buf[i] != pri[i]; };
     {  // the write ends at file_off + len: the file is at least that long, even if
        // its last bytes equal the pristine copy (zeros past the old EOF).
        // fallocate only ever grows the size (concurrent writers never shrink it).
@@ -669,10 +672,20 @@ int32_t do_write(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) 
     bool wm_ok = true;
     uint64_t i = 0, runs = 0;
     while (i < q.len) {
-      while (i < q.len && buf[i] == pri[i]) ++i;  // (a memcmp-by-words scan would be faster; pages are small)
+      if (bits) {  // skip unchanged 64-byte words whole
+        while (i < q.len && !(i & 63) && mw[i >> 6] == 0) i += 64;
+      }
+      while (i < q.len && !changed(i)) ++i;
       if (i >= q.len) break;
       uint64_t j = i;
-      while (j < q.len && buf[j] != pri[j]) ++j;
+      if (bits) {
+        while (j < q.len && !(j & 63) && j + 64 <= q.len && mw[j >> 6] == ~0ull) j += 64;
+      }
+      while (j < q.len && changed(j)) {
+        ++j;
+        if (bits && !(j & 63))
+          while (j + 64 <= q.len && mw[j >> 6] == ~0ull) j += 64;
+      }
       if (!wm && wm_ok) {
         wm = hfid_wmap(h, w, q.hfid, fd, q.file_off + q.len);
         wm_ok = wm != nullptr;
