@@ -226,7 +226,7 @@ typedef struct gfs_grep_params {
   uint64_t list_cap;    /* bytes of the list file (capacity) */
   uint64_t pair_cap;    /* (file, word) table slots (rounded up to a power of two) */
   uint64_t hit_cap;     /* hits to list in d_hits (0: none) */
-  uint32_t chunk;       /* work-item bytes, multiple of 16 */
+  uint32_t chunk;       /* work-item bytes, multiple of 16, at most 65472 (item + halos < 64 KiB: 16-bit offsets) */
   uint32_t grid;        /* persistent blocks */
   uint32_t block;       /* threads per block, multiple of 32, <= 256 */
   uint32_t keep_open;   /* 1: leave every file open after the run (warm re-runs skip the host) */

@@ -1042,7 +1042,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
                      const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
                      uint64_t* d_hits, uint64_t* d_summary) {
   if (!h || !dict_path || !list_path || !p || !d_work || !d_totals || !d_summary || p->max_files == 0 ||
-      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) || p->chunk > 65536 ||
+      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) || p->chunk + kPre + kHalo > 65536 ||  // u16 token offsets
       p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31))
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;

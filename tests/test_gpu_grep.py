@@ -104,3 +104,16 @@ def test_warp_item_scan_vs_oracle(g, shmdir, chunk, monkeypatch):
                  max_files=1024) as fs:
         out = fs.grep(c["dict"], c["list"], hits=True, chunk=chunk, grid=64)
     compare(out, ref)
+
+
+def test_max_chunk_and_rejected_chunk(g, shmdir):
+    """The largest item (65472 B: item + halos < 64 KiB, 16-bit token offsets) is
+    bit-exact; 65536 is rejected (it overflowed token offsets: wrong counts)."""
+    c = gen.c4_corpus(os.path.join(shmdir, "c4m"), seed=13, nfiles=120, total_bytes=4 << 20, nwords=2000)
+    ref = oracle.grep(c["dict"], c["list"], want_hits=True)
+    with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4,
+                 max_files=1024) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=True, chunk=65472, grid=64)
+        compare(out, ref)
+        with pytest.raises(g.GfsError):
+            fs.grep(c["dict"], c["list"], hits=False, chunk=65536, grid=64)

@@ -1,5 +1,7 @@
+# C4 grep timing sweep over (chunk, block) for the block scan (and optionally GFS_GREP_WARP=1)
 mkdir -p gpurun_out
 export RUNS=4
-python tools/grep_timing.py > gpurun_out/gt_base.log 2>&1
-for ch in 4096 8192; do GFS_GREP_WARP=1 CHUNK=$ch python tools/grep_timing.py > gpurun_out/gt_warp_$ch.log 2>&1; done
-GFS_GREP_WARP=1 CHUNK=4096 BLOCK=128 python tools/grep_timing.py > gpurun_out/gt_warp_4096_128.log 2>&1
+for cb in 32768:256 32768:128 16384:256 16384:128 8192:128 65536:256; do
+  ch=${cb%%:*}; bl=${cb##*:}
+  CHUNK=$ch BLOCK=$bl python tools/grep_timing.py 2>&1 | tail -1 >> gpurun_out/gt_sweep.log
+done
