@@ -1347,13 +1347,15 @@ __device__ __noinline__ int ensure_pristine(const gfs_ctx* c, Scratch& sc, uint3
     } else {
       uint32_t ns = 64;
       const uint64_t t0 = now_ns();
-      while (ld_acq(&c->f_pristine[f]) == GFS_PRISTINE_PENDING) {
+      uint32_t pv;
+      while ((pv = ld_acq(&c->f_pristine[f])) == GFS_PRISTINE_PENDING) {
         backoff(ns);
         if (timed_out(c, t0)) {
           atomicMin(&sc.err, -ETIMEDOUT);
           break;
         }
       }
+      if (pv == 0) atomicMin(&sc.err, -ENOMEM);  // its maker found no frame: never write without a pristine copy
     }
   }
   G::sync();
