@@ -160,7 +160,13 @@ def run_ours(args):
     import paper_conf_asplos_silbersteinfkw13_b200 as g
 
     ws, rank, local = dist_env()
-    if ws > 1:
+    if os.environ.get("GFS_BENCH_ONE_GPU") == "1":
+        # test mode for the multi-rank path on a one-GPU box: every rank on cuda:0, gloo
+        # (NCCL refuses two ranks on one GPU); never used for reported numbers
+        local = 0
+        if ws > 1:
+            dist.init_process_group("gloo")
+    elif ws > 1:
         dist.init_process_group("nccl", device_id=torch.device(f"cuda:{local}"))
     torch.cuda.set_device(local)
     dev = f"cuda:{local}"
