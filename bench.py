@@ -593,6 +593,8 @@ def c5_phase(args, torch, g, dev, stream, h2d, hbm, rank, ws, local, dist):
     root = "/dev/shm/gfs_bench_c5"
     os.makedirs(root, exist_ok=True)
     mine, peer = f"{root}/f_{rank}.bin", f"{root}/f_{(rank + 1) % ws}.bin"
+    if os.path.exists(mine):  # a write-once open does not truncate: start from no file
+        os.remove(mine)
     base = torch.from_numpy(np.random.default_rng(500 + rank).integers(0, 256, size=size, dtype=np.uint8)).to(dev)
     src = torch.empty_like(base)
     grid = 296
