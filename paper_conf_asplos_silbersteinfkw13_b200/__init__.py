@@ -21,7 +21,7 @@ COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", 
             "ring_wait", "busy", "stage_wait", "peer_fill", "bytes_peer", "peer_miss"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
                  "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns",
-                 "mapped_reads"]
+                 "mapped_reads", "open_vt_ns"]
 
 O_RDONLY = 0
 O_GWRONCE = 1

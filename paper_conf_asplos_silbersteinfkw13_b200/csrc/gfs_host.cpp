@@ -153,7 +153,7 @@ struct VersionTable {
 
 enum {
   HS_RPC = 0, HS_READ, HS_WRITE, HS_OPEN, HS_CLOSE, HS_TRUNC, HS_BYTES_H2D, HS_BYTES_D2H, HS_PREAD_NS,
-  HS_ERRORS, HS_MERGES, HS_BUSY_NS, HS_OPEN_NS, HS_OPEN_SYS_NS, HS_OPEN_PF_NS, HS_OPEN_TAB_NS, HS_MAPPED, HS_N
+  HS_ERRORS, HS_MERGES, HS_BUSY_NS, HS_OPEN_NS, HS_OPEN_SYS_NS, HS_OPEN_PF_NS, HS_OPEN_TAB_NS, HS_MAPPED, HS_OPEN_VT_NS, HS_N
 };
 
 }  // namespace
@@ -198,6 +198,24 @@ struct Worker {
   std::deque<uint32_t> fifo;                          // eviction order of fds
   std::unordered_map<std::string, int> dirfds;       // directory fds for openat()
   size_t cap = 1024;
+  // this worker's daemon counters (HS_*): one shared array took a contended
+  // atomic per counter per RPC (~9 per OPEN) and grew the per-OPEN cost with the
+  // thread count; gfs_host_stats sums the workers. Own-thread relaxed adds.
+  alignas(64) uint64_t hs[HS_N] = {};
+  void add(int k, uint64_t v) { __atomic_fetch_add(&hs[k], v, __ATOMIC_RELAXED); }
+};
+
+// Test-and-test-and-set lock for the host file table: its critical sections
+// are a few hundred nanoseconds of memory operations.
+struct SpinMutex {
+  std::atomic<bool> held{false};
+  void lock() {
+    for (;;) {
+      if (!held.exchange(true, std::memory_order_acquire)) return;
+      while (held.load(std::memory_order_relaxed)) cpu_relax();
+    }
+  }
+  void unlock() { held.store(false, std::memory_order_release); }
 };
 
 struct gfs_handle {
@@ -216,7 +234,8 @@ struct gfs_handle {
   std::atomic<uint64_t> frontier{0};  // one past the highest ticket whose request has arrived
   std::atomic<int64_t> last_arrival_ns{0};  // steady-clock time of the latest request
   std::atomic<bool> running{false};
-  std::mutex fd_mu;  // protects files / free_hfids
+  SpinMutex fd_mu;  // protects files / free_hfids (short sections: a futex sleep/wake per contended
+                    // acquisition cost ~2 us per OPEN with 12 workers)
   std::vector<HostFile> files;
   uint32_t nmapped = 0;
   uint32_t nwmapped = 0;
@@ -248,7 +267,7 @@ int cuda_err(cudaError_t e) {
   } while (0)
 
 uint32_t alloc_hfid(gfs_handle* h, HostFile&& f, uint32_t* gen_out) {
-  std::lock_guard<std::mutex> g(h->fd_mu);
+  std::lock_guard<SpinMutex> g(h->fd_mu);
   f.live = true;
   uint32_t id;
   if (!h->free_hfids.empty()) {
@@ -267,7 +286,7 @@ uint32_t alloc_hfid(gfs_handle* h, HostFile&& f, uint32_t* gen_out) {
 
 // Metadata of a live hfid.
 bool hfid_meta(gfs_handle* h, uint32_t id, HostFile* out) {
-  std::lock_guard<std::mutex> g(h->fd_mu);
+  std::lock_guard<SpinMutex> g(h->fd_mu);
   if (id >= h->files.size() || !h->files[id].live) return false;
   *out = h->files[id];
   return true;
@@ -278,7 +297,7 @@ void free_hfid(gfs_handle* h, uint32_t id) {
   uint64_t map_len = 0;
   uint8_t* wmap = nullptr;
   {
-    std::lock_guard<std::mutex> g(h->fd_mu);
+    std::lock_guard<SpinMutex> g(h->fd_mu);
     if (id >= h->files.size() || !h->files[id].live) return;
     const uint32_t gen = h->files[id].gen + 1;
     map = h->files[id].map;
@@ -396,14 +415,22 @@ void w_cache(Worker& w, uint32_t id, int fd, uint32_t gen) {
 
 // This worker's fd for hfid (opened by path on first use). -errno on failure.
 int w_fd(gfs_handle* h, Worker& w, uint32_t id) {
-  HostFile m;
-  if (!hfid_meta(h, id, &m)) return -EBADF;
   auto it = w.fds.find(id);
-  if (it != w.fds.end()) {
-    if (it->second.gen == m.gen) return it->second.fd;
+  if (it != w.fds.end()) {  // hot path: compare the generation only (no copy of the path under the lock)
+    uint32_t gen = 0;
+    bool live = false;
+    {
+      std::lock_guard<SpinMutex> g(h->fd_mu);
+      live = id < h->files.size() && h->files[id].live;
+      if (live) gen = h->files[id].gen;
+    }
+    if (!live) return -EBADF;
+    if (it->second.gen == gen) return it->second.fd;
     ::close(it->second.fd);  // the hfid was recycled for another file
     w.fds.erase(it);
   }
+  HostFile m;
+  if (!hfid_meta(h, id, &m)) return -EBADF;
   const int fd = w_open_path(w, m.path, (m.mode & GFS_O_WRITABLE) ? O_RDWR : O_RDONLY);
   if (fd < 0) return -errno;
   struct stat st;
@@ -427,7 +454,7 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
   auto tk0 = std::chrono::steady_clock::now();
   auto lap = [&](int k) {
     const auto t = std::chrono::steady_clock::now();
-    h->hs[k] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(t - tk0).count();
+    w.add(k, (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(t - tk0).count());
     tk0 = t;
   };
   gfs_rpc_resp* rs = h->resp_h + slot;
@@ -454,8 +481,8 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
     if (r >= 0) {
       if ((uint64_t)r < n) memset(buf + r, 0, n - (size_t)r);
       rs->pad[0] = n;
-      h->hs[HS_READ]++;
-      h->hs[HS_BYTES_H2D] += n;
+      w.add(HS_READ, 1);
+      w.add(HS_BYTES_H2D, n);
     }
   }
   lap(HS_OPEN_PF_NS);
@@ -488,6 +515,7 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
     hfid = alloc_hfid(h, std::move(f), &gen);
     w_cache(w, hfid, fd, gen);
   }
+  lap(HS_OPEN_TAB_NS);
   rs->size = (int64_t)st.st_size;
   rs->version = h->vt.get(st.st_dev, st.st_ino);
   rs->ino = st.st_ino;
@@ -495,8 +523,8 @@ int32_t do_open(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) {
   rs->mtime_ns = (int64_t)st.st_mtim.tv_sec * 1000000000ll + st.st_mtim.tv_nsec;
   rs->hfid = hfid;
   rs->status = 0;
-  h->hs[HS_OPEN]++;
-  lap(HS_OPEN_TAB_NS);
+  w.add(HS_OPEN, 1);
+  lap(HS_OPEN_VT_NS);
   return 0;
 }
 
@@ -506,7 +534,7 @@ const uint8_t* hfid_map(gfs_handle* h, Worker& w, uint32_t id, uint64_t* map_len
   uint64_t size;
   uint32_t gen;
   {
-    std::lock_guard<std::mutex> g(h->fd_mu);
+    std::lock_guard<SpinMutex> g(h->fd_mu);
     if (id >= h->files.size() || !h->files[id].live) return nullptr;
     HostFile& f = h->files[id];
     if (f.map) {
@@ -524,7 +552,7 @@ const uint8_t* hfid_map(gfs_handle* h, Worker& w, uint32_t id, uint64_t* map_len
   void* p = mmap(nullptr, size, PROT_READ, MAP_SHARED, fd, 0);
   if (p == MAP_FAILED) return nullptr;
   install_sigbus();
-  std::lock_guard<std::mutex> g(h->fd_mu);
+  std::lock_guard<SpinMutex> g(h->fd_mu);
   HostFile& f = h->files[id];
   if (!f.live || f.gen != gen || f.map) {
     munmap(p, size);
@@ -544,7 +572,7 @@ int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   uint64_t map_len = 0;
   const uint8_t* map = hfid_map(h, w, q.hfid, &map_len);
   if (!map) {  // a write-once file read back (re-opened read-only): its write mapping, below the known size
-    std::lock_guard<std::mutex> g(h->fd_mu);
+    std::lock_guard<SpinMutex> g(h->fd_mu);
     if (q.hfid < h->files.size() && h->files[q.hfid].live && h->files[q.hfid].wmap) {
       map = h->files[q.hfid].wmap;
       map_len = h->files[q.hfid].wsize;
@@ -553,18 +581,18 @@ int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   int64_t n = -1;
   if (map && q.file_off + q.len <= map_len && map_copy(buf, map, q.file_off, q.len)) {
     n = q.len;
-    h->hs[HS_MAPPED]++;
+    w.add(HS_MAPPED, 1);
   } else {
     const int fd = w_fd(h, w, q.hfid);
     if (fd < 0) return fd;
     n = pread_full(fd, buf, q.len, q.file_off);
   }
-  h->hs[HS_PREAD_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
-                            std::chrono::steady_clock::now() - t0).count();
+  w.add(HS_PREAD_NS, (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
+                            std::chrono::steady_clock::now() - t0).count());
   if (n < 0) return (int32_t)n;
   if ((uint64_t)n < q.len) memset(buf + n, 0, q.len - (size_t)n);  // host file shrank: zeros (R4)
-  h->hs[HS_READ]++;
-  h->hs[HS_BYTES_H2D] += q.len;
+  w.add(HS_READ, 1);
+  w.add(HS_BYTES_H2D, q.len);
   return (int32_t)q.len;
 }
 
@@ -592,7 +620,7 @@ uint8_t* hfid_wmap(gfs_handle* h, Worker& w, uint32_t id, int fd, uint64_t end) 
   uint32_t gen;
   bool map_it = false;
   {
-    std::lock_guard<std::mutex> g(h->fd_mu);
+    std::lock_guard<SpinMutex> g(h->fd_mu);
     if (id >= h->files.size() || !h->files[id].live) return nullptr;
     HostFile& f = h->files[id];
     map = f.wmap;
@@ -610,7 +638,7 @@ uint8_t* hfid_wmap(gfs_handle* h, Worker& w, uint32_t id, int fd, uint64_t end) 
     install_sigbus();
     struct stat st;
     wsize = fstat(fd, &st) == 0 ? (uint64_t)st.st_size : 0;
-    std::lock_guard<std::mutex> g(h->fd_mu);
+    std::lock_guard<SpinMutex> g(h->fd_mu);
     HostFile& f = h->files[id];
     if (!f.live || f.gen != gen || f.wmap) {
       munmap(p, kWMapReserve);
@@ -631,7 +659,7 @@ uint8_t* hfid_wmap(gfs_handle* h, Worker& w, uint32_t id, int fd, uint64_t end) 
     // back as zeros, ~5% of first-iteration C5 runs)
     if ((uint64_t)st.st_size < end && fallocate(fd, 0, 0, (off_t)end) != 0) return nullptr;
     const uint64_t now = (uint64_t)st.st_size > end ? (uint64_t)st.st_size : end;
-    std::lock_guard<std::mutex> g(h->fd_mu);
+    std::lock_guard<SpinMutex> g(h->fd_mu);
     HostFile& f = h->files[id];
     if (!f.live || f.gen != gen) return nullptr;
     if (f.wsize < now) f.wsize = now;
@@ -695,12 +723,12 @@ int32_t do_write(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) 
         if (r < 0) return (int32_t)r;
       }
       ++runs;
-      h->hs[HS_BYTES_D2H] += j - i;
+      w.add(HS_BYTES_D2H, j - i);
       i = j;
     }
     h->resp_h[slot].version = h->vt.bump(f.dev, f.ino);
-    h->hs[HS_WRITE]++;
-    h->hs[HS_MERGES]++;
+    w.add(HS_WRITE, 1);
+    w.add(HS_MERGES, 1);
     return (int32_t)q.len;
   }
   if (!(q.flags & GFS_WF_FULL)) {
@@ -710,20 +738,20 @@ int32_t do_write(gfs_handle* h, Worker& w, uint32_t slot, const gfs_rpc_req& q) 
     if (r < 0) return (int32_t)r;
     for (uint32_t i = 0; i < q.len; ++i)
       if (buf[i] == 0) buf[i] = w.merge[i];
-    h->hs[HS_MERGES]++;
+    w.add(HS_MERGES, 1);
   }
   uint8_t* wm = hfid_wmap(h, w, q.hfid, fd, q.file_off + q.len);
   if (!(wm && map_store(wm, buf, q.file_off, q.len))) {
     int64_t r = pwrite_full(fd, buf, q.len, q.file_off);
     if (r < 0) return (int32_t)r;
   } else {
-    h->hs[HS_MAPPED]++;
+    w.add(HS_MAPPED, 1);
   }
   // the version this write-back left the file at: the GPU records it as the
   // entry's synced version (peer fill); stored before completion
   h->resp_h[slot].version = h->vt.bump(f.dev, f.ino);
-  h->hs[HS_WRITE]++;
-  h->hs[HS_BYTES_D2H] += q.len;
+  w.add(HS_WRITE, 1);
+  w.add(HS_BYTES_D2H, q.len);
   return (int32_t)q.len;
 }
 
@@ -790,12 +818,12 @@ void worker_loop(gfs_handle* h, int wi) {
       case GFS_OP_WRITE: res = do_write(h, w, slot, q); break;
       case GFS_OP_OPEN:
         res = do_open(h, w, slot, q);
-        h->hs[HS_OPEN_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
-                                 std::chrono::steady_clock::now() - tb).count();
+        w.add(HS_OPEN_NS, (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
+                                 std::chrono::steady_clock::now() - tb).count());
         break;
       case GFS_OP_CLOSE:
         free_hfid(h, q.hfid);
-        h->hs[HS_CLOSE]++;
+        w.add(HS_CLOSE, 1);
         res = 0;
         break;
       case GFS_OP_TRUNC: {
@@ -803,17 +831,17 @@ void worker_loop(gfs_handle* h, int wi) {
         const int fd = hfid_meta(h, q.hfid, &f) ? w_fd(h, w, q.hfid) : -EBADF;
         res = fd < 0 ? fd : (ftruncate(fd, (off_t)q.arg) == 0 ? 0 : -errno);
         if (res == 0) h->vt.bump(f.dev, f.ino);
-        h->hs[HS_TRUNC]++;
+        w.add(HS_TRUNC, 1);
         break;
       }
       case GFS_OP_NOP: res = 0; break;
       default: res = -ENOSYS;
     }
-    if (res < 0) h->hs[HS_ERRORS]++;
-    h->hs[HS_RPC]++;
+    if (res < 0) w.add(HS_ERRORS, 1);
+    w.add(HS_RPC, 1);
     complete(h, slot, t, res);
-    h->hs[HS_BUSY_NS] += (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
-                             std::chrono::steady_clock::now() - tb).count();
+    w.add(HS_BUSY_NS, (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
+                             std::chrono::steady_clock::now() - tb).count());
   }
   for (auto& kv : w.fds) ::close(kv.second.fd);  // this worker's private table
   for (auto& kv : w.dirfds) ::close(kv.second);
@@ -1145,7 +1173,11 @@ GFS_API int gfs_stats(gfs_handle* h, uint64_t* out, int n, int reset) {
 
 GFS_API int gfs_host_stats(gfs_handle* h, uint64_t* out, int n) {
   if (!h || !out) return -EINVAL;
-  for (int i = 0; i < n && i < HS_N; ++i) out[i] = h->hs[i].load();
+  for (int i = 0; i < n && i < HS_N; ++i) {
+    uint64_t v = h->hs[i].load();
+    for (const Worker& w : h->workers) v += __atomic_load_n(&w.hs[i], __ATOMIC_RELAXED);
+    out[i] = v;
+  }
   return HS_N;
 }
 

@@ -10,7 +10,7 @@ block = int(os.environ.get("BLOCK", "256"))
 runs = int(os.environ.get("RUNS", "6"))
 c = gen.c4_corpus(f"/dev/shm/gfs_bench_c4_{nf}_{mib}", seed=4, nfiles=nf, total_bytes=mib << 20, nwords=58000)
 s = torch.cuda.Stream()
-with g.GpuFS(cache_bytes=4 << 30, page_size=64 << 10, daemon_threads=12, max_files=1 << 16) as fs:
+with g.GpuFS(cache_bytes=4 << 30, page_size=64 << 10, daemon_threads=int(os.environ.get("DAEMON", "12")), max_files=1 << 16) as fs:
     state = fs.grep_state(c["dict"], c["list"], keep_open=True, rec_cap=1 << 24, chunk=chunk, block=block)
     for it in range(runs):
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
@@ -21,5 +21,9 @@ with g.GpuFS(cache_bytes=4 << 30, page_size=64 << 10, daemon_threads=12, max_fil
             e1.record(s)
         s.synchronize()
         summ = dict(zip(g.GREP_SUMMARY, (int(x) for x in state["summary"].cpu().numpy())))
+        if it == 0 and os.environ.get("HOST_STATS"):
+            hs = fs.host_stats()
+            print({k: hs[k] for k in ("open", "read", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns", "open_vt_ns",
+                                      "pread_ns", "busy_ns", "bytes_h2d")}, fs.stats()["rpc_open"], flush=True)
         print(f"chunk={chunk} block={block}", "cold" if it == 0 else "warm", f"{e0.elapsed_time(e1):.3f} ms",
               summ["err"], summ["nhits"], summ["nrecords"], summ["digest_xor"], flush=True)
