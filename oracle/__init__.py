@@ -54,6 +54,7 @@ def lib():
             L.orc_cache_read.argtypes = [p, ci, u64, u64, p]; L.orc_cache_read.restype = i64
             L.orc_cache_mmap_copy.argtypes = [p, ci, u64, u64, p]; L.orc_cache_mmap_copy.restype = i64
             L.orc_cache_write.argtypes = [p, ci, u64, u64, p]; L.orc_cache_write.restype = i64
+            L.orc_cache_mmap_write.argtypes = [p, ci, u64, u64, p, ci]; L.orc_cache_mmap_write.restype = i64
             L.orc_cache_fsync.argtypes = [p, ci]; L.orc_cache_fsync.restype = ci
             L.orc_cache_ftruncate.argtypes = [p, ci, u64]; L.orc_cache_ftruncate.restype = ci
             L.orc_cache_stats.argtypes = [p, p]; L.orc_cache_stats.restype = None
@@ -105,10 +106,12 @@ def checksum(path, off: int, length: int) -> int:
 
 
 class PageCache:
-    """Page-cache model of P:L587-622 (O1/O2). flags: 0 = O_RDONLY, 1 = O_GWRONCE."""
+    """Page-cache model of P:L587-622 (O1/O2). flags: 0 = O_RDONLY, 1 = O_GWRONCE,
+    2 = O_RDWR (pristine copy + diff write-back)."""
 
     RDONLY = 0
     GWRONCE = 1
+    RDWR = 2
 
     def __init__(self, page_size: int, capacity_pages: int):
         self.h = lib().orc_cache_new(page_size, capacity_pages)
@@ -145,6 +148,12 @@ class PageCache:
     def write(self, fd, off, data) -> int:
         a = np.frombuffer(bytes(data), dtype=np.uint8).copy()
         return _check(lib().orc_cache_write(self.h, fd, off, len(a), _ptr(a) if len(a) else None))
+
+    def mmap_write(self, fd, off, data, msync=False) -> int:
+        """Writable gmmap of an O_RDWR file + stores (+ gmsync); returns the mapped prefix length."""
+        a = np.frombuffer(bytes(data), dtype=np.uint8).copy()
+        return _check(lib().orc_cache_mmap_write(self.h, fd, off, len(a), _ptr(a) if len(a) else None,
+                                                 1 if msync else 0))
 
     def fsync(self, fd):
         return _check(lib().orc_cache_fsync(self.h, fd))

@@ -132,7 +132,10 @@ ORC_API int64_t orc_checksum(const char* path, uint64_t off, uint64_t len, uint6
 // (§3.1), gclose without write-back,
 // gfsync writing back dirty pages (Tab.1), and lazy
 // invalidation on re-open (§4.4) keyed by a per-path version that
-// every write-back bumps (the user-space stand-in for WRAPFS, R7).
+// every write-back bumps (the user-space stand-in for WRAPFS, R7),
+// and O_RDWR write sharing: pages are fetched, a pristine copy is
+// preserved before the first local write (R21), and write-back sends
+// only the bytes where the working copy differs from the pristine one.
 // ---------------------------------------------------------------------------
 namespace {
 
@@ -153,6 +156,7 @@ struct OFile {
   int hfd = -1;
   uint64_t size = 0;       // snapshot at first gopen, max written end if writable
   bool gwronce = false;
+  bool rdwr = false;
   uint64_t version = 0;
   uint64_t uid = 0;
   int refs = 0;
@@ -163,6 +167,7 @@ struct OPage {
   bool dirty = false;
   uint64_t lo = 0, hi = 0;    // dirty byte range within the page
   uint64_t written = 0;       // bytes written into the page by gwrite
+  std::vector<uint8_t> pristine;  // O_RDWR: copy taken before the first local write (empty: none)
   int file = -1;
 };
 
@@ -183,6 +188,25 @@ int64_t writeback(OCache* c, OPage& pg, const PKey& k) {
   OFile& f = c->files[pg.file];
   uint64_t base = k.second * c->P;
   uint64_t n = pg.hi - pg.lo;
+  if (!pg.pristine.empty()) {
+    // O_RDWR: "diff" the working and pristine copies and write
+    // only the bytes that differ; the file is extended to the write's end.
+    struct stat st;
+    if (fstat(f.hfd, &st) != 0) return -errno;
+    if ((uint64_t)st.st_size < base + pg.hi && ftruncate(f.hfd, (off_t)(base + pg.hi)) != 0) return -errno;
+    for (uint64_t i = pg.lo; i < pg.hi; ++i) {
+      if (pg.data[i] == pg.pristine[i]) continue;
+      int64_t r = pwrite_full(f.hfd, &pg.data[i], 1, base + i);
+      if (r < 0) return r;
+    }
+    pg.pristine.clear();
+    pg.dirty = false;
+    pg.lo = pg.hi = pg.written = 0;
+    c->writebacks++;
+    version_bump(f.path);
+    f.version = version_of(f.path);
+    return 0;
+  }
   std::vector<uint8_t> out(pg.data.begin() + pg.lo, pg.data.begin() + pg.hi);
   if (pg.written < n) {
     // Not every byte of [lo,hi) was written: "diff against zeros"
@@ -293,34 +317,37 @@ ORC_API void orc_cache_free(void* h) {
   delete c;
 }
 
-// flags: 0 = O_RDONLY, 1 = O_GWRONCE.
+// flags: 0 = O_RDONLY, 1 = O_GWRONCE, 2 = O_RDWR.
 ORC_API int orc_cache_open(void* h, const char* path, int flags) {
   OCache* c = (OCache*)h;
-  bool gw = (flags & 1) != 0;
+  if (flags < 0 || flags > 2) return -EINVAL;
+  const bool rw = flags == 2;
+  bool gw = flags == 1;
   std::string p(path);
   for (size_t i = 0; i < c->files.size(); ++i) {
     OFile& f = c->files[i];
     if (f.path != p) continue;
     if (f.refs > 0) {
       // Already open on this GPU: the fd is shared.
-      if (f.gwronce != gw) return -EBUSY;  // one writer at a time
+      if (f.gwronce != gw || f.rdwr != rw) return -EBUSY;  // one mode at a time
       f.refs++;
       return (int)i;
     }
     // Closed-file cache: re-open validates.
     struct stat st;
     if (stat(path, &st) != 0) return -errno;
-    bool stale = gw || f.gwronce || version_of(p) != f.version || (uint64_t)st.st_size != f.size;
+    bool stale = gw || rw || f.gwronce || f.rdwr || version_of(p) != f.version || (uint64_t)st.st_size != f.size;
     if (stale) {
       int64_t r = drop_file_pages(c, f.uid);
       if (r < 0) return (int)r;
       if (f.hfd >= 0) close(f.hfd);
-      f.hfd = gw ? open(path, O_RDWR | O_CREAT, 0644) : open(path, O_RDONLY);
+      f.hfd = (gw || rw) ? open(path, O_RDWR | O_CREAT, 0644) : open(path, O_RDONLY);
       if (f.hfd < 0) return -errno;
       if (fstat(f.hfd, &st) != 0) return -errno;
       f.uid = c->next_uid++;
-      f.size = gw ? (uint64_t)st.st_size : (uint64_t)st.st_size;
+      f.size = (uint64_t)st.st_size;
       f.gwronce = gw;
+      f.rdwr = rw;
       f.version = version_of(p);
     }
     f.refs = 1;
@@ -328,12 +355,13 @@ ORC_API int orc_cache_open(void* h, const char* path, int flags) {
   }
   OFile f;
   f.path = p;
-  f.hfd = gw ? open(path, O_RDWR | O_CREAT, 0644) : open(path, O_RDONLY);
+  f.hfd = (gw || rw) ? open(path, O_RDWR | O_CREAT, 0644) : open(path, O_RDONLY);
   if (f.hfd < 0) return -errno;
   struct stat st;
   if (fstat(f.hfd, &st) != 0) return -errno;
   f.size = (uint64_t)st.st_size;
   f.gwronce = gw;
+  f.rdwr = rw;
   f.version = version_of(p);
   f.uid = c->next_uid++;
   f.refs = 1;
@@ -389,12 +417,14 @@ ORC_API int64_t orc_cache_mmap_copy(void* h, int fd, uint64_t off, uint64_t len,
 }
 
 // gwrite on an O_GWRONCE file: pages are zero-initialised, never fetched;
-// the dirty range and written-byte count are tracked; size grows.
+// on an O_RDWR file: pages are fetched and keep a pristine copy from before
+// the first local write. The dirty range and written-byte count are tracked;
+// size grows.
 ORC_API int64_t orc_cache_write(void* h, int fd, uint64_t off, uint64_t len, const uint8_t* in) {
   OCache* c = (OCache*)h;
   if (fd < 0 || (size_t)fd >= c->files.size() || c->files[fd].refs <= 0) return -EBADF;
   OFile& f = c->files[fd];
-  if (!f.gwronce) return -EBADF;
+  if (!f.gwronce && !f.rdwr) return -EBADF;
   uint64_t done = 0;
   while (done < len) {
     uint64_t o = off + done;
@@ -403,6 +433,7 @@ ORC_API int64_t orc_cache_write(void* h, int fd, uint64_t off, uint64_t len, con
     int64_t err = 0;
     OPage* pg = get_page(c, fd, p, &err);
     if (!pg) return err;
+    if (f.rdwr && pg->pristine.empty()) pg->pristine = pg->data;
     memcpy(pg->data.data() + in_off, in + done, take);
     if (!pg->dirty) {
       pg->dirty = true;
@@ -417,6 +448,47 @@ ORC_API int64_t orc_cache_write(void* h, int fd, uint64_t off, uint64_t len, con
   }
   f.size = std::max(f.size, off + len);
   return (int64_t)len;
+}
+
+// A writable gmmap of an O_RDWR file, stores through it, and (do_msync) gmsync
+// (Tab.1, R22/R23): the mapped prefix m = min(len, P - off%P,
+// S - off) is written; the page keeps its pristine copy and the range is
+// dirty; gmsync writes the page's diff back now and makes the written-back
+// state the new pristine copy (the page stays dirty: the mapping may be
+// written again). Returns m.
+ORC_API int64_t orc_cache_mmap_write(void* h, int fd, uint64_t off, uint64_t len, const uint8_t* in,
+                                     int do_msync) {
+  OCache* c = (OCache*)h;
+  if (fd < 0 || (size_t)fd >= c->files.size() || c->files[fd].refs <= 0) return -EBADF;
+  OFile& f = c->files[fd];
+  if (!f.rdwr) return -EBADF;
+  if (off >= f.size || len == 0) return 0;
+  const uint64_t p = off / c->P, in_off = off % c->P;
+  const uint64_t m = std::min(std::min(len, c->P - in_off), f.size - off);
+  int64_t err = 0;
+  OPage* pg = get_page(c, fd, p, &err);
+  if (!pg) return err;
+  if (pg->pristine.empty()) pg->pristine = pg->data;
+  memcpy(pg->data.data() + in_off, in, m);
+  if (!pg->dirty) {
+    pg->dirty = true;
+    pg->lo = in_off;
+    pg->hi = in_off + m;
+  } else {
+    pg->lo = std::min<uint64_t>(pg->lo, in_off);
+    pg->hi = std::max<uint64_t>(pg->hi, in_off + m);
+  }
+  if (do_msync) {
+    const PKey k(f.uid, p);
+    const uint64_t lo = pg->lo, hi = pg->hi;
+    int64_t r = writeback(c, *pg, k);
+    if (r < 0) return r;
+    pg->pristine = pg->data;  // the written-back state
+    pg->dirty = true;         // still mapped writable: keep the range
+    pg->lo = lo;
+    pg->hi = hi;
+  }
+  return (int64_t)m;
 }
 
 // gfsync: write back every dirty page of the file.

@@ -11,6 +11,8 @@ import os
 import numpy as np
 import pytest
 
+import oracle
+
 pytestmark = [pytest.mark.gpu, pytest.mark.timeout(600)]
 RDWR = 2
 
@@ -103,6 +105,18 @@ def test_rdwr_two_writers_share_pages(g, shmdir):
         A.unpin(fa)
         B.unpin(fb)
     assert host(path) == apply(orig, wa + wb)
+    # the oracle's page-cache model (two caches, same writes) leaves the same file
+    q = os.path.join(shmdir, "share_oracle.bin")
+    open(q, "wb").write(orig)
+    oa, ob = oracle.PageCache(P, 32), oracle.PageCache(P, 32)
+    qa, qb = oa.open(q, oracle.PageCache.RDWR), ob.open(q, oracle.PageCache.RDWR)
+    for o, b in wa:
+        oa.write(qa, o, b)
+    for o, b in wb:
+        ob.write(qb, o, b)
+    oa.fsync(qa)
+    ob.fsync(qb)
+    assert host(path) == host(q)
 
 
 def test_rdwr_host_change_not_reverted(g, shmdir):
@@ -170,6 +184,19 @@ def test_rdwr_mmap_gmsync(g, shmdir):
         assert fs.gfsync(path, flags=RDWR) == 0
         fs.unpin(fd)
     assert host(path) == apply(orig, w1 + [(3000, b"\x11" * 8)] + w2)
+    q = os.path.join(shmdir, "mm_oracle.bin")
+    open(q, "wb").write(orig)
+    pc = oracle.PageCache(P, 32)
+    qf = pc.open(q, oracle.PageCache.RDWR)
+    for o, b in w1:
+        pc.mmap_write(qf, o, b, msync=True)
+    with open(q, "r+b") as f:
+        f.seek(3000)
+        f.write(b"\x11" * 8)
+    for o, b in w2:
+        pc.mmap_write(qf, o, b, msync=False)
+    pc.fsync(qf)
+    assert host(path) == host(q)
 
 
 def test_rdwr_mode_rules(g, shmdir):

@@ -111,3 +111,97 @@ def test_ftruncate(shmdir):
     pc.write(fd, 0, b"\x01\x02")
     pc.fsync(fd)
     assert host_bytes(p) == b"\x01\x02" and pc.size(fd) == 2
+
+
+# ---- O_RDWR diff-and-merge (NEXT-4) pinned to the definition of
+# workspace consistency with disjoint writers: the original bytes with every
+# writer's bytes laid over them (built here from the buffers, read back with
+# plain host reads).
+def overlay(base: bytes, writes):
+    out = bytearray(base)
+    for o, b in writes:
+        if o + len(b) > len(out):
+            out.extend(b"\x00" * (o + len(b) - len(out)))
+        out[o:o + len(b)] = b
+    return bytes(out)
+
+
+def test_rdwr_reads_own_writes_and_syncs_only_changes(shmdir):
+    p = os.path.join(shmdir, "rw.bin")
+    orig = rnd(3 * 4096 + 100, 40)
+    open(p, "wb").write(orig)
+    pc = oracle.PageCache(4096, 16)
+    fd = pc.open(p, oracle.PageCache.RDWR)
+    w = [(10, rnd(50, 41)), (4090, rnd(20, 42)), (3 * 4096 + 150, rnd(30, 43))]  # straddle, past EOF
+    for o, b in w:
+        assert pc.write(fd, o, b) == len(b)
+    want = overlay(orig, w)
+    assert pc.read(fd, 0, len(want)) == want          # own writes visible before any sync
+    assert host_bytes(p) == orig
+    with open(p, "r+b") as f:                         # another writer, bytes this cache never wrote
+        f.seek(2000)
+        f.write(b"\x07" * 9)
+    assert pc.fsync(fd) == 0
+    assert host_bytes(p) == overlay(want, [(2000, b"\x07" * 9)])
+
+
+def test_rdwr_two_writers_false_sharing(shmdir):
+    p = os.path.join(shmdir, "share.bin")
+    orig = rnd(2 * 4096, 44)
+    open(p, "wb").write(orig)
+    a, b = oracle.PageCache(4096, 8), oracle.PageCache(4096, 8)
+    fa, fb = a.open(p, oracle.PageCache.RDWR), b.open(p, oracle.PageCache.RDWR)
+    wa = [(o, rnd(16, 100 + o)) for o in range(0, 2 * 4096, 64)]
+    wb = [(o + 32, rnd(16, 200 + o)) for o in range(0, 2 * 4096, 64)]
+    for o, d in wa:
+        a.write(fa, o, d)
+    for o, d in wb:
+        b.write(fb, o, d)
+    assert a.fsync(fa) == 0 and b.fsync(fb) == 0
+    assert host_bytes(p) == overlay(orig, wa + wb)
+
+
+def test_rdwr_eviction_writes_back_diffs(shmdir):
+    p = os.path.join(shmdir, "ev.bin")
+    orig = rnd(20 * 4096, 45)
+    open(p, "wb").write(orig)
+    pc = oracle.PageCache(4096, 3)
+    fd = pc.open(p, oracle.PageCache.RDWR)
+    w = [(k * 4096 + 7, rnd(33, 300 + k)) for k in range(20)]
+    for o, d in w:
+        pc.write(fd, o, d)
+    assert pc.stats()["evictions"] >= 17
+    assert pc.fsync(fd) == 0
+    assert host_bytes(p) == overlay(orig, w)
+
+
+def test_rdwr_mmap_write_and_msync(shmdir):
+    p = os.path.join(shmdir, "mm.bin")
+    orig = rnd(2 * 4096, 46)
+    open(p, "wb").write(orig)
+    pc = oracle.PageCache(4096, 8)
+    fd = pc.open(p, oracle.PageCache.RDWR)
+    assert pc.mmap_write(fd, 4000, rnd(200, 47), msync=True) == 96      # prefix of one page
+    w1 = [(4000, rnd(200, 47)[:96])]
+    assert host_bytes(p) == overlay(orig, w1)                             # gmsync reached the host
+    with open(p, "r+b") as f:
+        f.seek(3000)
+        f.write(b"\x05" * 4)
+    assert pc.mmap_write(fd, 3990, b"\x09" * 5, msync=False) == 5
+    assert pc.fsync(fd) == 0
+    assert host_bytes(p) == overlay(orig, w1 + [(3000, b"\x05" * 4), (3990, b"\x09" * 5)])
+
+
+def test_rdwr_mode_conflict(shmdir):
+    p = os.path.join(shmdir, "m.bin")
+    open(p, "wb").write(rnd(100, 48))
+    pc = oracle.PageCache(4096, 4)
+    pc.open(p, oracle.PageCache.RDWR)
+    with pytest.raises(oracle.OracleError):
+        pc.open(p, oracle.PageCache.RDONLY)        # one mode at a time while open
+    ro = oracle.PageCache(4096, 4)
+    fd = ro.open(p, oracle.PageCache.RDONLY)
+    with pytest.raises(oracle.OracleError):
+        ro.write(fd, 0, b"x")                      # read-only files are never written
+    with pytest.raises(oracle.OracleError):
+        ro.mmap_write(fd, 0, b"x")                 # nor mapped writable
