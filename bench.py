@@ -726,7 +726,7 @@ def rdwr_phase(args, torch, g, dev):
         fds = [c.pin(path, flags=g.O_RDWR) for c in caches]
         for k, c in enumerate(caches):
             mine = offs[k::2]
-            data = np.concatenate([new[int(o):int(o) + blk] for o in mine]).tobytes()
+            data = torch.from_numpy(np.concatenate([new[int(o):int(o) + blk] for o in mine])).to(dev)
             e = [torch.cuda.Event(enable_timing=True) for _ in range(4)]
             torch.cuda.synchronize()
             e[0].record()
@@ -754,8 +754,9 @@ def rdwr_phase(args, torch, g, dev):
             "gwrite_GBps": round(half / (float(np.mean(times["gwrite"])) * 1e-3) / 1e9, 3),
             "gfsync_GBps": round(half / (float(np.mean(times["gfsync"])) * 1e-3) / 1e9, 3),
             "parity": bool(ok), "writebacks": [x["writeback"] for x in st], "misses": [x["miss"] for x in st],
-            "note": "gwrite includes the page fetches (O_RDWR reads pages) and pristine copies; gfsync moves "
-                    "working + pristine ranges over PCIe and the host writes only changed bytes"}
+            "note": "source bytes resident in HBM; gwrite includes the page fetches (O_RDWR reads pages) and "
+                    "pristine copies; gfsync diffs on the GPU, moves bytes + mask over PCIe, the host writes "
+                    "only changed bytes"}
 
 
 def c5_local_peer(args, torch, g, fs, path, size, P, grid, dev, stream, scratch, out):

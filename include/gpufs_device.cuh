@@ -2108,7 +2108,13 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
     const uint32_t B = nthr < 32 ? (uint32_t)nthr : 32u;
     uint32_t ns = 256;
     const uint64_t t0 = now_ns();
-    for (uint64_t pb = 0; pb < np;) {
+    // Blocks syncing one file together start at different batches (rotated by
+    // block id) so the dirty pages spread over them instead of the first
+    // blocks claiming most of them; every block still visits every batch.
+    const uint64_t nbat = (np + B - 1) / B;
+    const uint64_t b0 = nbat ? block_linear() % nbat : 0;
+    for (uint64_t bi = 0; bi < nbat;) {
+      const uint64_t pb = ((b0 + bi) % nbat) * B;
       const uint32_t cnt = (uint32_t)((np - pb) < B ? (np - pb) : B);
       if (tid == 0) sc.busy = 0;
       __syncthreads();
@@ -2187,7 +2193,7 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
       }
       __syncthreads();
       if (!sc.busy) {
-        pb += B;
+        ++bi;
         ns = 256;
       } else {  // some page of the batch found no staging slot: back off, redo the batch
         if (tid == 0 && timed_out(c, t0)) atomicMin(&sc.err, -ETIMEDOUT);

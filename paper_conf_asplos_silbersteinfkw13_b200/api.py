@@ -185,8 +185,11 @@ class GpuFS:
         n = len(offs)
         if srcoff is None:
             srcoff = np.concatenate([[0], np.cumsum(lens)[:-1]]).astype(np.uint64) if n else np.zeros(0, np.uint64)
-        src = np.frombuffer(bytes(data), dtype=np.uint8) if len(data) else np.zeros(1, np.uint8)
-        d_src = self._dev(src)
+        if hasattr(data, "data_ptr"):  # a device uint8 tensor already resident (no upload)
+            d_src = data
+        else:
+            src = np.frombuffer(bytes(data), dtype=np.uint8) if len(data) else np.zeros(1, np.uint8)
+            d_src = self._dev(src)
         d_off = self._dev(offs.view(np.int64))
         d_len = self._dev(lens.view(np.int64))
         d_srcoff = self._dev(np.asarray(srcoff, np.uint64).view(np.int64))
