@@ -55,7 +55,36 @@ class Clocks:
         self._stop = threading.Event()
         self._th = None
 
+    def _nvml_handle(self):
+        """In-process NVML (no nvidia-smi process per sample competing with the daemon's
+        workers for host cores); the device found by PCI bus id (CUDA ordinals may be remapped)."""
+        try:
+            import pynvml
+            import torch
+            pynvml.nvmlInit()
+            pr = torch.cuda.get_device_properties(self.index)
+            bus = f"{pr.pci_domain_id:08x}:{pr.pci_bus_id:02x}:{pr.pci_device_id:02x}.0"
+            return pynvml, pynvml.nvmlDeviceGetHandleByPciBusId(bus)
+        except Exception:
+            return None, None
+
     def __enter__(self):
+        nv, hd = self._nvml_handle()
+
+        def run_nvml():
+            act = lambda m, bit: "Active" if m & bit else "Not Active"
+            while not self._stop.is_set():
+                try:
+                    m = nv.nvmlDeviceGetCurrentClocksEventReasons(hd) \
+                        if hasattr(nv, "nvmlDeviceGetCurrentClocksEventReasons") \
+                        else nv.nvmlDeviceGetCurrentClocksThrottleReasons(hd)
+                    self.samples.append([str(nv.nvmlDeviceGetClockInfo(hd, nv.NVML_CLOCK_SM)),
+                                         str(nv.nvmlDeviceGetMaxClockInfo(hd, nv.NVML_CLOCK_SM)),
+                                         act(m, 0x8), act(m, 0x40), act(m, 0x20), act(m, 0x4)])
+                except Exception:
+                    pass
+                self._stop.wait(0.2)
+
         def run():
             q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,"
                  "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
@@ -71,7 +100,7 @@ class Clocks:
                     pass
                 self._stop.wait(0.2)
 
-        self._th = threading.Thread(target=run, daemon=True)
+        self._th = threading.Thread(target=run_nvml if hd is not None else run, daemon=True)
         self._th.start()
         return self
 
