@@ -428,6 +428,7 @@ __device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64
     resp_out->hfid = r->hfid;
     resp_out->status = r->status;
     resp_out->pad[0] = r->pad[0];  // OPEN: bytes of page 0 prefetched into the staging slot
+    resp_out->pad[1] = r->pad[1];  // OPEN: device address of the registered file mapping (0: none)
   }
   st_rel64(&c->ack[slot], (uint64_t)(t + 1));
   return res;
@@ -1019,13 +1020,18 @@ __device__ __forceinline__ void peer_release(const gfs_ctx* c, int code) {
   const gfs_peer& P = c->peers[(uint32_t)code >> kPeerFrameBits];
   a64_add_sys(&P.f_state[(uint32_t)code & ((1u << kPeerFrameBits) - 1u)], kRefDec);
 }
-// Lk.stage / Scratch.stage: >= 0 staging slot, -1 nothing to pull, <= -2 peer frame
+// Lk.stage / Scratch.stage: >= 0 staging slot, -1 nothing to pull, kStageZC
+// the file's registered host mapping (zero-copy), other values <= -2 a peer frame
+constexpr int kStageZC = -0x7FFFFFFF;
 __device__ __forceinline__ int peer_stage(int code) { return -2 - code; }
 __device__ __forceinline__ int stage_peer(int stage) { return -2 - stage; }
-__device__ __forceinline__ const uint8_t* fill_src(const gfs_ctx* c, int stage) {
+__device__ __forceinline__ const uint8_t* fill_src(const gfs_ctx* c, int stage, const FileSnap& fs,
+                                                   uint64_t page) {
+  if (stage == kStageZC) return (const uint8_t*)ld_rlx64(&c->files[fs.fdx].zc) + (page << c->page_shift);
   return stage >= 0 ? stage_ptr(c, stage) : peer_frame_ptr(c, stage_peer(stage));
 }
 __device__ __forceinline__ void fill_src_free(const gfs_ctx* c, int stage) {
+  if (stage == kStageZC) return;
   if (stage >= 0) stage_free(c, stage);
   else peer_release(c, stage_peer(stage));
 }
@@ -1111,9 +1117,14 @@ __device__ __noinline__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint
     const uint32_t nb = (fs.oflags & GFS_O_GWRONCE) ? 0u : (uint32_t)(rem < c->page_size ? rem : c->page_size);
     // A peer GPU's cache may hold the page (NEXT-1): then no staging slot
     // and no RPC; `st` names the peer frame (held) instead.
-    const int pc = (nb && c->npeers) ? peer_take(c, fs, page, nb) : -1;
+    // A registered host mapping of the file (gfs_register_file): the block pulls
+    // the page straight from the host page cache, no RPC and no staging slot.
+    const bool zc = nb && ld_rlx64(&c->files[fs.fdx].zc) != 0;
+    const int pc = (nb && !zc && c->npeers) ? peer_take(c, fs, page, nb) : -1;
     int st = -1;
-    if (pc >= 0) {
+    if (zc) {
+      st = kStageZC;
+    } else if (pc >= 0) {
       st = peer_stage(pc);
     } else if (nb) {
       st = stage_alloc(c, false);
@@ -1146,6 +1157,14 @@ __device__ __noinline__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint
     out.fill = 1;
     if (fs.oflags & GFS_O_GWRONCE) {
       ctr(c, GFS_C_ZERO_FILL);
+      break;
+    }
+    if (zc) {  // the block pulls from the registered mapping over PCIe
+      out.stage = st;
+      out.nbytes = nb;
+      ctr(c, GFS_C_MISS);
+      ctr(c, GFS_C_ZC_FILL);
+      ctr(c, GFS_C_BYTES_H2D, nb);
       break;
     }
     if (pc >= 0) {  // the block copies the peer frame over NVLink
@@ -1233,8 +1252,8 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
     if (pull) {  // fill the frames this block installed: staging -> frame over PCIe, or peer frame -> frame
       for (uint32_t i = 0; i < cnt; ++i)
         if (sc.frame[i] >= 0 && sc.fill[i] && sc.stage[i] != -1) {
-          block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), fill_src(c, sc.stage[i]), sc.nbytes[i],
-                                      tid, nthr);
+          block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), fill_src(c, sc.stage[i], fs, pb + i),
+                                      sc.nbytes[i], tid, nthr);
           // a writable page past the old EOF reads (and diffs) as zeros, not a previous tenant's bytes
           if ((fs.oflags & GFS_O_RDWR) && sc.nbytes[i] < c->page_size)
             block_zero(frame_ptr(c, (uint32_t)sc.frame[i]) + sc.nbytes[i], c->page_size - sc.nbytes[i], tid, nthr);
@@ -1552,6 +1571,7 @@ __device__ int new_incarnation(const gfs_ctx* c, gfs_file* e, uint32_t flags, co
   e->mtime_ns = rs.mtime_ns;
   e->oflags = flags;
   e->synced_version = 0;
+  e->zc = (flags & GFS_O_WRITABLE) ? 0ull : rs.pad[1];  // zero-copy source for read-only opens
   return 0;
 }
 
@@ -1701,6 +1721,7 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, uint32_t n, uint6
                         rs.dev == e->dev && rs.mtime_ns == e->mtime_ns;
       if (same) {
         e->hfid = rs.hfid;
+        e->zc = rs.pad[1];
         ctr(c, GFS_C_REOPEN_VALID);
       } else {
         tree_free(c, old.root, old.height);  // old frames become orphans (tier 0)

@@ -85,6 +85,8 @@ typedef struct gfs_file {
   uint32_t pad;
   uint64_t synced_version; /* O_GWRONCE: host version after this cache's last write-back
                               (peer fill); 0 = none */
+  uint64_t zc;             /* device address of the host file's registered page-cache mapping
+                              (gfs_register_file; misses pull from it directly), 0 = none */
 } gfs_file;
 
 /* ---- RPC (§4.3) -------------------------------------------- */
@@ -162,6 +164,7 @@ enum {
   GFS_C_PEER_FILL,      /* misses filled from a peer GPU's cache (NVLink) instead of the host */
   GFS_C_BYTES_PEER,     /* bytes copied from peer caches */
   GFS_C_PEER_MISS,      /* misses for which no peer held a usable copy */
+  GFS_C_ZC_FILL,        /* misses filled straight from a registered file mapping (no RPC) */
   GFS_C_NCOUNTERS
 };
 

@@ -18,7 +18,7 @@ LIB_PATH = os.path.join(_PKG, "libgpufs.so")
 COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", "writeback", "rpc",
             "rpc_open", "rpc_read", "rpc_write", "bytes_h2d", "bytes_d2h", "open_fast", "reopen_valid",
             "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
-            "ring_wait", "busy", "stage_wait", "peer_fill", "bytes_peer", "peer_miss"]
+            "ring_wait", "busy", "stage_wait", "peer_fill", "bytes_peer", "peer_miss", "zc_fill"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
                  "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns",
                  "mapped_reads", "open_vt_ns"]
@@ -86,6 +86,7 @@ def lib():
             "gfs_host_stats": ([P, P, I], I),
             "gfs_info": ([P, P, I], I),
             "gfs_export": ([P, ctypes.POINTER(gfs_export_desc)], I),
+            "gfs_register_file": ([P, CS], I),
             "gfs_attach_peer": ([P, ctypes.POINTER(gfs_export_desc)], I),
             "gfs_run_gread": ([P, P, CS, I, U32, P, P, P, P, P, U32, U32, U32], I),
             "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
@@ -165,6 +166,11 @@ def gfs_info(h: int) -> dict:
     _ck(lib().gfs_info(h, a, 9), "gfs_info")
     return dict(zip(["page_size", "nframes", "max_files", "max_nodes", "ring_slots", "daemon_threads",
                      "staging_slots", "host_next_ticket", "device_ring_tail"], (int(x) for x in a)))
+
+
+def gfs_register_file(h: int, path) -> int:
+    """Zero-copy misses for `path` (include/gpufs.h gfs_register_file)."""
+    return _ck(lib().gfs_register_file(h, _b(path)), "gfs_register_file")
 
 
 def gfs_export(h: int) -> bytes:

@@ -64,6 +64,12 @@ class GpuFS:
     def info(self) -> dict:
         return gfs_info(self.h)
 
+    def register_file(self, path) -> int:
+        """Map `path` for zero-copy misses (gfs_register_file): O_RDONLY misses of it
+        are pulled straight from the host page cache, without RPCs."""
+        from . import gfs_register_file
+        return gfs_register_file(self.h, path)
+
     # peer caches (NEXT-1) -------------------------------------------------
     def export(self) -> bytes:
         """Describe this cache for attach_peer in another process or GpuFS (gfs_export)."""

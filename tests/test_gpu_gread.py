@@ -249,3 +249,32 @@ def test_few_staging_slots_many_missing_pages(g, shmdir):
             assert err == 0 and s == oracle.checksum(path, 0, size)
         st = fs.stats()
     assert st["timeout"] == 0 and st["stage_wait"] > 0
+
+
+@pytest.mark.parametrize("P", [65536, 1 << 21])
+def test_zero_copy_registered_file(g, shmdir, P):
+    """gfs_register_file: misses of the registered file pull straight from the host
+    page cache (no READ RPC); every byte still equals pread (oracle), under
+    eviction churn; an unregistered file in the same cache still uses RPCs."""
+    size = 40 * P + 777
+    path = gen.splitmix_file(os.path.join(shmdir, "zc.bin"), size, seed=41)
+    other = gen.splitmix_file(os.path.join(shmdir, "plain.bin"), 5 * P + 3, seed=42)
+    with _fs(g, cache_bytes=12 * P, page_size=P) as fs:
+        assert fs.register_file(path) == 0
+        fs.stats(reset=True)
+        offs, lens = gen.random_calls(43, 300, size, 3 * P, page_size=P)
+        ret, dst, dstoff = fs.gread_calls(path, offs, lens, grid=4)
+        for i, (o, l) in enumerate(zip(offs.tolist(), lens.tolist())):
+            exp = oracle.pread(path, size, o, l)
+            assert ret[i] == len(exp)
+            assert dst[int(dstoff[i]):int(dstoff[i]) + len(exp)].tobytes() == exp, i
+        s, err = fs.seqread(path, size - size % 8, P, grid=4)
+        assert err == 0 and s == oracle.checksum(path, 0, size - size % 8)
+        st = fs.stats()
+        assert st["zc_fill"] > 0 and st["rpc_read"] == 0 and st["evict"] > 0, st
+        ret, dst, dstoff = fs.gread_calls(other, [0], [5 * P + 3], grid=1)
+        assert dst[:5 * P + 3].tobytes() == open(other, "rb").read()
+        assert fs.stats()["rpc_read"] > 0
+    with pytest.raises(g.GfsError):
+        with _fs(g, cache_bytes=4 * P, page_size=P) as fs2:
+            fs2.register_file(os.path.join(shmdir, "missing.bin"))
