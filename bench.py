@@ -587,6 +587,30 @@ def matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local):
         err = int(state["err"][0].item())
         y = state["y"].cpu().numpy().astype(np.float64)
         st = fs.stats()
+        # the same product with the matrix file registered (zero-copy misses, §4.3 of DESIGN.md)
+        zc = None
+        if not args.no_zc:
+            try:
+                t0 = time.perf_counter()
+                fs.register_file(m["A"])
+                reg_s = time.perf_counter() - t0
+                zts = []
+                for it in range(3):
+                    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                    with torch.cuda.stream(stream):
+                        e0.record(stream)
+                        state = fs.matvec(m["A"], m["x"], ypath, rows, cols, stream=stream, sync=False,
+                                          state=state)
+                        e1.record(stream)
+                        stream.synchronize()
+                    zts.append(e0.elapsed_time(e1))
+                zy = state["y"].cpu().numpy().astype(np.float64)
+                zms = float(np.median(zts))
+                zc = {"GBps": round(nbytes / (zms * 1e-3) / 1e9, 3),
+                      "frac_h2d": round(nbytes / (zms * 1e-3) / 1e9 / h2d, 4), "register_s": round(reg_s, 2),
+                      "y_equal_rpc_path": bool(np.array_equal(zy, y)) and int(state["err"][0].item()) == 0}
+            except Exception as e:
+                zc = {"unavailable": str(e)[:200]}
     ms = float(np.median(ts))
     gbs = nbytes / (ms * 1e-3) / 1e9
     rng = np.random.default_rng(0)
@@ -601,6 +625,8 @@ def matvec_phase(args, torch, g, gen, dev, stream, h2d, rank, local):
                         "frac": round(gbs / h2d, 4)},
            "max_rel_err_sampled_rows": relerr, "parity_ok": relerr <= 1e-5 and np.array_equal(yh, y),
            "misses": st["miss"], "evictions": st["evict"]}
+    if zc:
+        out["zero_copy"] = zc
     if not args.no_cpu:
         t0 = time.perf_counter()
         n = min(rows, 2048)
