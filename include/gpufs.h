@@ -237,11 +237,17 @@ typedef struct gfs_grep_params {
   uint64_t list_cap;    /* bytes of the list file (capacity) */
   uint64_t pair_cap;    /* (file, word) table slots (rounded up to a power of two) */
   uint64_t hit_cap;     /* hits to list in d_hits (0: none) */
-  uint32_t chunk;       /* work-item bytes, multiple of 16, at most 65472 (item + halos < 64 KiB: 16-bit offsets) */
-  uint32_t grid;        /* persistent blocks */
+  uint32_t chunk;       /* work-item bytes: a file larger than this is split into chunks of it;
+                           multiple of 16, at most 65472 (item + halos < 64 KiB: 16-bit offsets) */
+  uint32_t grid;        /* persistent blocks (at most one per resident block slot) */
   uint32_t block;       /* threads per block, multiple of 32, <= 256 */
-  uint32_t keep_open;   /* 1: leave every file open after the run (warm re-runs skip the host) */
+  uint32_t keep_open;   /* 1: leave every file (and the dictionary and list) open after the run:
+                           warm re-runs skip the host (no close-to-open revalidation) */
   uint64_t corpus_cap;  /* bytes of all listed files (capacity, sizes the work-item map) */
+  const uint32_t* file_ids; /* device array: file i of the list is reported as file_ids[i] in
+                           records, hits and the digest (e.g. a shard's global indices); NULL:
+                           the list index i */
+  uint64_t rec_cap;     /* records the work area can stage (>= the records found, else -ENOSPC) */
 } gfs_grep_params;
 
 /* Device scratch bytes gfs_grep needs for these parameters. */
@@ -256,7 +262,10 @@ uint64_t gfs_grep_work_bytes(const gfs_grep_params* p);
  *   d_summary[0..9]     = nrecords, nhits, digest_sum, digest_xor, nfiles, nwords,
  *                         corpus bytes, error (0 or -errno), nhits_listed, nitems.
  * The digest is sum and xor over hits of splitmix64(splitmix64(splitmix64(f)+off)+k)
- * (order independent). File index = position among the list's non-empty lines. */
+ * (order independent). File index = position among the list's non-empty lines, or
+ * file_ids[position] when given. The work area also carries state across runs
+ * with the same d_work (an empty (file, word) table, the held dictionary and
+ * list with keep_open): reuse it only with the same parameters. */
 int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
              const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
              uint64_t* d_hits, uint64_t* d_summary);
@@ -274,6 +283,14 @@ int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* lis
 int gfs_matvec(gfs_handle* h, void* stream, const char* a_path, const char* x_path, const char* y_path,
                uint64_t rows, uint64_t cols, float* d_x, float* d_y, int64_t* d_err, uint32_t grid,
                uint32_t block);
+
+/* The same for the row block [row0, row0 + nrows) of A (a rank's shard in the
+ * multi-GPU C3): y_path and d_y receive those nrows values only
+ * (y_path's element i is y_{row0+i}). -EINVAL if the range is empty or
+ * exceeds rows. */
+int gfs_matvec_rows(gfs_handle* h, void* stream, const char* a_path, const char* x_path, const char* y_path,
+                    uint64_t rows, uint64_t cols, uint64_t row0, uint64_t nrows, float* d_x, float* d_y,
+                    int64_t* d_err, uint32_t grid, uint32_t block);
 
 #ifdef __cplusplus
 }

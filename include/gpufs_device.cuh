@@ -1755,6 +1755,35 @@ __device__ int close_leader(const gfs_ctx* c, int fd) {
   return 0;  // no write-back
 }
 
+// Snapshot for a caller that holds `fd` open through a gopen ordered before
+// the call (so the entry cannot change meanwhile): relaxed L2 loads only. An
+// acquire compiles to LDG.STRONG + CCTL.IVALL, which drops the SM's whole L1
+// (e.g. a consumer's L1-cached lookup tables) on every call.
+__device__ __forceinline__ bool snap_fd_rlx(const gfs_ctx* c, int fd, FileSnap* s) {
+  if (fd < 0 || (uint32_t)fd >= c->max_files) return false;
+  const gfs_file* e = c->files + fd;
+  // all loads issued together (one L2 round trip); the state is checked after
+  const uint32_t sr = ld_rlx(&e->sr);
+  s->fdx = (uint32_t)fd;
+  s->uid = ld_rlx(&e->uid);
+  s->root = ld_rlx(&e->root);
+  s->height = ld_rlx(&e->height);
+  s->hfid = ld_rlx(&e->hfid);
+  s->oflags = ld_rlx(&e->oflags);
+  s->size = ld_rlx64((const uint64_t*)&e->size);
+  return (sr >> 24) == GFS_FS_OPEN && (sr & 0xFFFFFF) != 0;
+}
+
+// The head and tail bytes of one co-aligned span that tma_span() leaves out,
+// copied by the calling thread alone (L2 loads: the frame may be refilled).
+__device__ __forceinline__ void lane_edges(uint8_t* dst, const uint8_t* src, uint32_t n) {
+  const uint32_t h0 = (16u - ((uint32_t)(uintptr_t)src & 15u)) & 15u;
+  const uint32_t head = h0 < n ? h0 : n;
+  const uint32_t mid = (n - head) & ~15u;
+  for (uint32_t i = 0; i < head; ++i) dst[i] = __ldcg(src + i);
+  for (uint32_t i = head + mid; i < n; ++i) dst[i] = __ldcg(src + i);
+}
+
 }  // namespace
 }  // namespace detail
 
@@ -2017,6 +2046,146 @@ __device__ inline int64_t gfstat_size_warp(const gfs_ctx* c, int fd) {
 }
 __device__ inline int64_t gread_warp(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
   return gread_t<detail::WarpGroup>(c, fd, off, len, dst);
+}
+
+namespace detail {
+namespace {
+// gread_lanes' one-request-at-a-time remainder, out of line so the callers'
+// fast path keeps its registers.
+__device__ __noinline__ int64_t gread_warp_slow(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+  return gread_t<WarpGroup>(c, fd, off, len, dst);
+}
+}  // namespace
+}  // namespace detail
+
+// gread_lanes: a warp-collective VECTORED gread (an extension in the spirit of
+// P:L449-452's "data transfer scheduling"): every lane of the calling warp
+// passes its OWN request (fd, off, len, dst) and receives its own result, with
+// gread's pread semantics (EOF at the size snapshot). A
+// lane passing len 0 (or fd < 0) takes no part and gets 0 (-EBADF for a bad
+// fd with len > 0).
+//
+// Requests whose span covers at most two pages that are all cache hits, and
+// whose destination is shared memory co-aligned with the offset
+// ((dst - off) % 16 == 0), are served in one round: the lanes look their pages
+// up at the same time (lock-free, one atomic per page), lane 0
+// arms the warp's mbarrier with the total byte count, every lane issues its
+// own TMA bulk copies (cp.async.bulk) and copies its <16-byte edges, and the
+// warp waits ONCE for all of them — 32 requests cost about one request's
+// latency. Every other request (a miss, a longer span, a global destination)
+// is served one at a time by gread_warp, so misses keep their full semantics
+// (RPC, eviction). Each fd must be held open by the caller through a gopen
+// ordered before the call (the snapshot uses relaxed loads only, so the SM's
+// L1 survives the call). Full warps only; uses the warp's scratch.
+//
+// Split phase (NEXT-2): gread_lanes_issue() returns once the hit
+// copies are IN FLIGHT (misses and other requests are complete by then);
+// gread_lanes_wait() waits for them and drops the page references. The
+// destination must not be touched in between; a warp has at most one issued,
+// unwaited request set, and makes no other warp-API call until it waits.
+// gread_lanes(...) is issue + wait.
+struct GreadLaneTicket {
+  int64_t ret;     // the lane's result
+  int32_t f0, f1;  // frames this lane holds until the wait (-1: none)
+  uint32_t total;  // (warp-uniform) bytes in flight on the warp's mbarrier; 0: nothing to wait for
+  uint32_t phase;  // (warp-uniform) the mbarrier phase to wait for
+};
+
+__device__ inline GreadLaneTicket gread_lanes_issue(const gfs_ctx* c, int fd, uint64_t off, uint64_t len,
+                                                    void* dst) {
+  using namespace detail;
+  Scratch& sc = WarpGroup::sc();
+  const int lane = block_tid() & 31;
+  const uint32_t shift = c->page_shift;
+  const uint64_t P = c->page_size;
+  __syncwarp();
+  GreadLaneTicket t{0, -1, -1, 0, 0};
+  FileSnap s;
+  if (len > 0 && fd >= 0) {
+    if (!snap_fd_rlx(c, fd, &s) || (s.oflags & GFS_O_GWRONCE)) t.ret = -EBADF;
+    else t.ret = off >= s.size ? 0 : (int64_t)(len < s.size - off ? len : s.size - off);
+  } else if (len > 0) {
+    t.ret = -EBADF;
+  }
+  uint32_t tx = 0, n0 = 0;
+  if (t.ret > 0 && t.ret < (1 << 20) && !(c->flags & GFS_F_LOCKED_TRAVERSAL) && __isShared(dst) &&
+      (((uintptr_t)dst - off) & 15) == 0) {
+    const uint64_t p0 = off >> shift, p1 = (off + (uint64_t)t.ret - 1) >> shift;
+    if (p1 - p0 <= 1) {
+      t.f0 = lookup_fast(c, s, p0, nullptr);
+      if (t.f0 >= 0 && p1 != p0) {
+        t.f1 = lookup_fast(c, s, p1, nullptr);
+        if (t.f1 < 0) {
+          r64_add_rlx(&c->f_state[t.f0], kRefDec);
+          t.f0 = -1;
+        }
+      }
+      if (t.f0 >= 0) {
+        const uint64_t in0 = off & (P - 1);
+        n0 = (uint32_t)(t.f1 >= 0 ? P - in0 : (uint64_t)t.ret);
+        tx = span_mid(frame_ptr(c, (uint32_t)t.f0) + in0, n0);
+        if (t.f1 >= 0) tx += span_mid(frame_ptr(c, (uint32_t)t.f1), (uint32_t)t.ret - n0);
+      }
+    }
+  }
+  const bool fast = t.f0 >= 0;
+  // the other requests first, one at a time, with the full warp-collective
+  // gread (it completes its own mbarrier phases before the fast copies arm one)
+  uint32_t slow = __ballot_sync(0xFFFFFFFFu, t.ret > 0 && !fast);
+  while (slow) {
+    const int src = __ffs(slow) - 1;
+    slow &= slow - 1;
+    const int sfd = __shfl_sync(0xFFFFFFFFu, fd, src);
+    const uint64_t soff = __shfl_sync(0xFFFFFFFFu, off, src);
+    const uint64_t slen = __shfl_sync(0xFFFFFFFFu, len, src);
+    void* sdst = (void*)__shfl_sync(0xFFFFFFFFu, (unsigned long long)(uintptr_t)dst, src);
+    const int64_t r = detail::gread_warp_slow(c, sfd, soff, slen, sdst);
+    if (lane == src) t.ret = r;
+  }
+  t.total = __reduce_add_sync(0xFFFFFFFFu, tx);
+  if (lane == 0) {
+    ensure_mbar<WarpGroup>(sc);
+    if (t.total) mbar_expect_tx(&sc.mbar, t.total);  // armed before any copy is issued
+  }
+  __syncwarp();
+  t.phase = sc.mbar_phase;
+  if (fast) {
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // earlier generic use of dst
+    const uint8_t* s0 = frame_ptr(c, (uint32_t)t.f0) + (off & (P - 1));
+    tma_span((uint8_t*)dst, s0, n0, &sc.mbar);
+    lane_edges((uint8_t*)dst, s0, n0);
+    if (t.f1 >= 0) {
+      const uint8_t* s1 = frame_ptr(c, (uint32_t)t.f1);
+      tma_span((uint8_t*)dst + n0, s1, (uint32_t)t.ret - n0, &sc.mbar);
+      lane_edges((uint8_t*)dst + n0, s1, (uint32_t)t.ret - n0);
+    }
+  }
+  __syncwarp();
+  if (lane == 0 && t.total) sc.mbar_phase = t.phase ^ 1u;  // this phase belongs to the ticket now
+  const uint32_t nfast = __popc(__ballot_sync(0xFFFFFFFFu, fast));
+  const uint32_t bfast = __reduce_add_sync(0xFFFFFFFFu, fast ? (uint32_t)t.ret : 0u);
+  if (lane == 0 && nfast) {
+    ctr(c, GFS_C_GREAD_CALLS, nfast);
+    ctr(c, GFS_C_GREAD_BYTES, bfast);
+  }
+  return t;
+}
+
+__device__ inline int64_t gread_lanes_wait(const gfs_ctx* c, GreadLaneTicket& t) {
+  using namespace detail;
+  Scratch& sc = WarpGroup::sc();
+  if (t.total) mbar_wait(&sc.mbar, t.phase);
+  __syncwarp();
+  if (t.f0 >= 0) frame_release(c, (uint32_t)t.f0);
+  if (t.f1 >= 0) frame_release(c, (uint32_t)t.f1);
+  t.f0 = t.f1 = -1;
+  t.total = 0;
+  return t.ret;
+}
+
+__device__ inline int64_t gread_lanes(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+  GreadLaneTicket t = gread_lanes_issue(c, fd, off, len, dst);
+  return gread_lanes_wait(c, t);
 }
 
 // gwrite: pwrite semantics on an O_GWRONCE file.

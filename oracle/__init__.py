@@ -46,6 +46,9 @@ def lib():
             L.orc_pread.argtypes = [cs, u64, u64, u64, p]; L.orc_pread.restype = i64
             L.orc_file_size.argtypes = [cs]; L.orc_file_size.restype = i64
             L.orc_checksum.argtypes = [cs, u64, u64, ctypes.POINTER(u64)]; L.orc_checksum.restype = i64
+            L.orc_checksum_mt.argtypes = [cs, u64, u64, ci, ctypes.POINTER(u64)]; L.orc_checksum_mt.restype = i64
+            L.orc_checksum_calls.argtypes = [cs, p, u64, u64, ci, ctypes.POINTER(u64)]
+            L.orc_checksum_calls.restype = i64
             L.orc_cache_new.argtypes = [u64, u64]; L.orc_cache_new.restype = p
             L.orc_cache_free.argtypes = [p]; L.orc_cache_free.restype = None
             L.orc_cache_open.argtypes = [p, cs, ci]; L.orc_cache_open.restype = ci
@@ -102,6 +105,23 @@ def checksum(path, off: int, length: int) -> int:
     """Position-weighted u64 checksum of file bytes [off, off+len) (R9)."""
     s = ctypes.c_uint64(0)
     _check(lib().orc_checksum(_b(path), off, length, ctypes.byref(s)))
+    return s.value
+
+
+def checksum_mt(path, off: int, length: int, nthreads: int = 0) -> int:
+    """The same checksum of [off, off+len), the range cut into nthreads pieces
+    (the sum is per byte, so pieces add up mod 2^64). nthreads 0: os.cpu_count()."""
+    s = ctypes.c_uint64(0)
+    _check(lib().orc_checksum_mt(_b(path), off, length, nthreads or os.cpu_count() or 1, ctypes.byref(s)))
+    return s.value
+
+
+def checksum_calls(path, offs, length: int, nthreads: int = 0) -> int:
+    """K4 consumer total: sum over calls i of checksum(path, offs[i], length) mod 2^64."""
+    o = np.ascontiguousarray(np.asarray(offs, dtype=np.uint64))
+    s = ctypes.c_uint64(0)
+    _check(lib().orc_checksum_calls(_b(path), _ptr(o) if o.size else None, o.size, length,
+                                    nthreads or os.cpu_count() or 1, ctypes.byref(s)))
     return s.value
 
 

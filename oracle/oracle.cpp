@@ -124,6 +124,75 @@ ORC_API int64_t orc_checksum(const char* path, uint64_t off, uint64_t len, uint6
   return 0;
 }
 
+// The same definition over a large range with T threads: the sum is over
+// bytes (each byte b at offset o adds (b << 8(o mod 8)) * (2(o div 8) + 1)),
+// so [off, off+len) is cut into T contiguous pieces, each summed by
+// orc_checksum above, and the pieces' sums are added mod 2^64. Used to check
+// the C2 sweep at its full size (8 GiB) in bench.py.
+ORC_API int64_t orc_checksum_mt(const char* path, uint64_t off, uint64_t len, int nthreads, uint64_t* out_sum) {
+  if (nthreads < 1) nthreads = 1;
+  std::vector<uint64_t> part(nthreads, 0);
+  std::vector<int64_t> rc(nthreads, 0);
+  std::vector<std::thread> th;
+  const uint64_t per = (len + nthreads - 1) / nthreads;
+  for (int t = 0; t < nthreads; ++t)
+    th.emplace_back([&, t]() {
+      const uint64_t a = std::min(len, per * (uint64_t)t), b = std::min(len, a + per);
+      if (b > a) rc[t] = orc_checksum(path, off + a, b - a, &part[t]);
+    });
+  for (auto& x : th) x.join();
+  uint64_t sum = 0;
+  for (int t = 0; t < nthreads; ++t) {
+    if (rc[t] < 0) return rc[t];
+    sum += part[t];
+  }
+  *out_sum = sum;
+  return 0;
+}
+
+// K4: the consumer adds the checksum of every chunk it reads;
+// the expected total is the sum over calls i of checksum(offs[i], len) — each
+// call's bytes read with pread, calls split over T threads.
+ORC_API int64_t orc_checksum_calls(const char* path, const uint64_t* offs, uint64_t ncalls, uint64_t len,
+                                   int nthreads, uint64_t* out_sum) {
+  if (nthreads < 1) nthreads = 1;
+  std::vector<uint64_t> part(nthreads, 0);
+  std::vector<int64_t> rc(nthreads, 0);
+  std::vector<std::thread> th;
+  for (int t = 0; t < nthreads; ++t)
+    th.emplace_back([&, t]() {
+      int fd = open(path, O_RDONLY);
+      if (fd < 0) {
+        rc[t] = -errno;
+        return;
+      }
+      std::vector<uint8_t> buf(len + 1);
+      uint64_t sum = 0;
+      for (uint64_t i = (uint64_t)t; i < ncalls; i += (uint64_t)nthreads) {
+        const int64_t r = pread_full(fd, buf.data(), len, offs[i]);
+        if (r < 0) {
+          rc[t] = r;
+          break;
+        }
+        if ((uint64_t)r < len) memset(buf.data() + r, 0, len - (uint64_t)r);
+        for (uint64_t k = 0; k < len; ++k) {
+          const uint64_t o = offs[i] + k;
+          sum += ((uint64_t)buf[k] << (8 * (o & 7))) * (2 * (o >> 3) + 1);
+        }
+      }
+      close(fd);
+      part[t] = sum;
+    });
+  for (auto& x : th) x.join();
+  uint64_t sum = 0;
+  for (int t = 0; t < nthreads; ++t) {
+    if (rc[t] < 0) return rc[t];
+    sum += part[t];
+  }
+  *out_sum = sum;
+  return 0;
+}
+
 // ---------------------------------------------------------------------------
 // Page-cache model (O1/O2): the simple buffer cache of P:L587-622 §4.2 with
 // per-file page lookup, an LRU of capacity C pages (the north star's

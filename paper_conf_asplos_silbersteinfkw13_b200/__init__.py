@@ -49,7 +49,7 @@ class gfs_grep_params(ctypes.Structure):
     _fields_ = [("max_files", ctypes.c_uint32), ("max_words", ctypes.c_uint32), ("list_cap", ctypes.c_uint64),
                 ("pair_cap", ctypes.c_uint64), ("hit_cap", ctypes.c_uint64), ("chunk", ctypes.c_uint32),
                 ("grid", ctypes.c_uint32), ("block", ctypes.c_uint32), ("keep_open", ctypes.c_uint32),
-                ("corpus_cap", ctypes.c_uint64)]
+                ("corpus_cap", ctypes.c_uint64), ("file_ids", ctypes.c_void_p), ("rec_cap", ctypes.c_uint64)]
 
 
 class gfs_export_desc(ctypes.Structure):
@@ -99,6 +99,7 @@ def lib():
             "gfs_grep_work_bytes": ([ctypes.POINTER(gfs_grep_params)], U64),
             "gfs_grep": ([P, P, CS, CS, ctypes.POINTER(gfs_grep_params), P, P, U64, P, P, P], I),
             "gfs_matvec": ([P, P, CS, CS, CS, U64, U64, P, P, P, U32, U32], I),
+            "gfs_matvec_rows": ([P, P, CS, CS, CS, U64, U64, U64, U64, P, P, P, U32, U32], I),
         }
         for name, (args, res) in sig.items():
             fn = getattr(L, name)
@@ -240,6 +241,11 @@ def gfs_grep(h, stream, dict_path, list_path, p: gfs_grep_params, d_work, d_rec,
 def gfs_matvec(h, stream, a_path, x_path, y_path, rows, cols, d_x, d_y, d_err, grid, block):
     return _ck(lib().gfs_matvec(h, stream, _b(a_path), _b(x_path), _b(y_path), rows, cols, d_x, d_y, d_err, grid,
                                 block), "gfs_matvec")
+
+
+def gfs_matvec_rows(h, stream, a_path, x_path, y_path, rows, cols, row0, nrows, d_x, d_y, d_err, grid, block):
+    return _ck(lib().gfs_matvec_rows(h, stream, _b(a_path), _b(x_path), _b(y_path), rows, cols, row0, nrows, d_x,
+                                     d_y, d_err, grid, block), "gfs_matvec_rows")
 
 
 from . import build  # noqa: E402,F401

@@ -224,9 +224,10 @@ class GpuFS:
 
     # grep -w ------------------------------------------------------------------
     def grep_state(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
-                   pair_cap=1 << 24, hit_cap=None, corpus_cap=1 << 34, rec_cap=1 << 22):
+                   pair_cap=1 << 24, hit_cap=None, corpus_cap=1 << 34, rec_cap=1 << 22, file_ids=None):
         """Device buffers of one grep configuration (allocated once, reused by grep(state=...)).
-        Capacities come from file metadata (stat), never from file contents."""
+        Capacities come from file metadata (stat), never from file contents. file_ids: optional
+        per-list-line ids reported instead of the line index (e.g. a shard's global file indices)."""
         import os
         torch = _torch()
         from . import gfs_grep_params, gfs_grep_work_bytes
@@ -235,7 +236,12 @@ class GpuFS:
         lbytes = os.path.getsize(list_path)
         p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
                             pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 1 << 20, block=block,
-                            keep_open=1 if keep_open else 0, corpus_cap=corpus_cap)
+                            keep_open=1 if keep_open else 0, corpus_cap=corpus_cap, rec_cap=rec_cap)
+        d_ids = None
+        if file_ids is not None:
+            d_ids = torch.as_tensor(np.ascontiguousarray(np.asarray(file_ids, dtype=np.uint32)).view(np.int32),
+                                    device=dev)
+            p.file_ids = d_ids.data_ptr()
         if hits:
             p.hit_cap = hit_cap if hit_cap is not None else 1 << 22
         work = torch.empty(gfs_grep_work_bytes(p), dtype=torch.uint8, device=dev)
@@ -243,11 +249,11 @@ class GpuFS:
         totals = torch.empty(nwords, dtype=torch.int64, device=dev)
         d_hits = torch.empty(2 * max(p.hit_cap, 1), dtype=torch.int64, device=dev) if hits else None
         summ = torch.zeros(10, dtype=torch.int64, device=dev)
-        return dict(p=p, work=work, rec=rec, rec_cap=rec_cap, totals=totals, hits=d_hits, summary=summ)
+        return dict(p=p, work=work, rec=rec, rec_cap=rec_cap, totals=totals, hits=d_hits, summary=summ, ids=d_ids)
 
     def grep(self, dict_path, list_path, hits=False, chunk=32768, grid=None, block=256, keep_open=False,
              pair_cap=1 << 24, hit_cap=None, stream=None, sync=True, state=None, corpus_cap=1 << 34,
-             rec_cap=1 << 22):
+             rec_cap=1 << 22, file_ids=None):
         """grep -w. Returns a dict with records (n,3) sorted by (file, word),
         totals, digest (sum, xor, nhits), hits (n,3) sorted by (file, offset, word) if requested.
         With sync=False, only enqueues and returns the state (read it after synchronising).
@@ -257,7 +263,7 @@ class GpuFS:
         from . import GREP_SUMMARY, gfs_grep
         if state is None:
             state = self.grep_state(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap, hit_cap,
-                                    corpus_cap, rec_cap)
+                                    corpus_cap, rec_cap, file_ids)
         p = state["p"]
         s, sp = self._stream(stream)
         gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
@@ -269,7 +275,7 @@ class GpuFS:
         summ = dict(zip(GREP_SUMMARY, (int(x) for x in state["summary"].cpu().numpy())))
         if summ["err"] == -28 and pair_cap < (1 << 30):  # -ENOSPC: a table was too small
             return self.grep(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap * 4, hit_cap,
-                             stream, sync, None, corpus_cap * 4, max(rec_cap, summ["nrecords"]) * 2)
+                             stream, sync, None, corpus_cap * 4, max(rec_cap, summ["nrecords"]) * 2, file_ids)
         out = {"summary": summ}
         nrec = min(summ["nrecords"], state["rec_cap"])
         r = state["rec"][:3 * nrec].view(nrec, 3).cpu().numpy().astype(np.uint64)
@@ -288,22 +294,25 @@ class GpuFS:
         return out
 
     # mat-vec -------------------------------------------------------------------
-    def matvec(self, a_path, x_path, y_path, rows, cols, grid=None, block=256, stream=None, sync=True, state=None):
-        """y = A x through gmmap/gwrite/gfsync. Returns (y device tensor, err)."""
+    def matvec(self, a_path, x_path, y_path, rows, cols, grid=None, block=256, stream=None, sync=True, state=None,
+               row0=0, nrows=None):
+        """y = A x through gmmap/gwrite/gfsync for rows [row0, row0 + nrows) of A
+        (default: all). Returns (y device tensor, err)."""
         torch = _torch()
-        from . import gfs_matvec
+        from . import gfs_matvec_rows
         dev = f"cuda:{self.device}"
+        nrows = rows - row0 if nrows is None else nrows
         if grid is None:
-            grid = max(1, min(rows, 4 * 148))
-            while (rows + grid - 1) // grid * 4 > 160 * 1024:
+            grid = max(1, min(nrows, 4 * 148))
+            while (nrows + grid - 1) // grid * 4 > 160 * 1024:
                 grid *= 2
         if state is None:
             state = dict(x=torch.empty(cols, dtype=torch.float32, device=dev),
-                         y=torch.empty(rows, dtype=torch.float32, device=dev),
+                         y=torch.empty(nrows, dtype=torch.float32, device=dev),
                          err=torch.zeros(2, dtype=torch.int64, device=dev))
         s, sp = self._stream(stream)
-        gfs_matvec(self.h, sp, a_path, x_path, y_path, rows, cols, state["x"].data_ptr(), state["y"].data_ptr(),
-                   state["err"].data_ptr(), grid, block)
+        gfs_matvec_rows(self.h, sp, a_path, x_path, y_path, rows, cols, row0, nrows, state["x"].data_ptr(),
+                        state["y"].data_ptr(), state["err"].data_ptr(), grid, block)
         if not sync:
             return state
         s.synchronize()

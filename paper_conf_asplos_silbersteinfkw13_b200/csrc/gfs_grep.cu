@@ -11,24 +11,28 @@
 // against the brute-force oracle) but the work is proportional to the corpus:
 //   k_grep_dict   gread the dictionary, validate slots, build an open-addressing
 //                 hash table (L2-resident) keyed by a 64-bit token hash;
-//   k_grep_list_* gread the file list in chunks, count line starts per chunk,
-//                 scan, emit absolute paths (parallel over the list);
-//   k_grep_open   gopen every file once (first gopen goes to the host,
-//                 P:L370-372), record fd and size;
-//   k_grep_plan   exclusive scan of per-file work-item counts, item -> file map;
-//   k_grep_scan   persistent blocks pull items: a whole file when it fits one
-//                 item, else a chunk of it. gread brings the item plus a halo
-//                 into shared memory (TMA). Pass 1 classifies 32-byte stripes
-//                 into word-byte bit masks (SWAR, 4 bytes per op); pass 2 gives
-//                 each thread the tokens that start in its stripe: length from
-//                 the masks, bytes gathered as 8 zero-padded words, one 64-bit
-//                 hash, one probe of the (L2-resident) table, an exact 32-byte
-//                 compare on a fingerprint match. Counts per item in shared
-//                 memory; a whole-file item emits its (file, word, count)
-//                 records directly, chunks of large files merge through a
-//                 global (file, word) table;
+//   k_grep_list_* gread the file list, find the line starts (parallel over the
+//                 list), record each line's offset;
+//   k_grep_open   one warp per file builds its path from the list line, gopen
+//                 (the first gopen goes to the host), gfstat;
+//   k_grep_plan   exclusive scan of per-file work-item counts; k_grep_items
+//                 writes one 32-byte descriptor per item (a whole file when it
+//                 fits one item, else a chunk of it): one round trip per item;
+//   k_grep_scan   persistent blocks pull items. gread brings the item plus a
+//                 halo into shared memory (TMA). Pass 1 classifies 32-byte
+//                 stripes into word-byte bit masks (SWAR, 4 bytes per op); pass
+//                 2 gives each thread the tokens that start in its stripe:
+//                 length from the masks, bytes gathered as 8 zero-padded words,
+//                 one hash, one probe of the (L2-resident) table, an exact
+//                 32-byte compare on a fingerprint match. Counts per item in
+//                 shared memory; a whole-file item emits its (file, word,
+//                 count) records directly (into a record page the block
+//                 reserved), chunks of large files merge through a global
+//                 (file, word) table;
 //   k_grep_close  gclose every file (unless kept open for warm re-runs);
-//   k_grep_compact emit unique (file, word, count) records and word totals.
+//   k_grep_compact emit the merged records and their word totals, and leave
+//                 the (file, word) table empty for the next run;
+//   k_grep_pack_* pack the record pages into the caller's contiguous array.
 // Word bytes are [A-Za-z0-9_] (GNU grep -w under LC_ALL=C, R10).
 #include <cuda_runtime.h>
 #include <errno.h>
@@ -36,10 +40,12 @@
 #include <stdio.h>
 #include <stdlib.h>
 #include <string.h>
-#include <time.h>
+
+#include <string>
 
 #include "gpufs.h"
 #include "gpufs_device.cuh"
+#include "gfs_launch.h"
 
 #define GFS_API extern "C" __attribute__((visibility("default")))
 
@@ -48,14 +54,29 @@ using namespace gfs;
 namespace {
 
 constexpr uint32_t kMaxPath = GFS_MAX_PATH;
-constexpr uint32_t kHalo = 48;      // bytes after the chunk: a token starting inside may run 33 bytes
-constexpr uint32_t kPre = 16;       // bytes before the chunk (one needed for the boundary test)
+constexpr uint32_t kHalo = 48;      // bytes after a chunk: a token starting inside may run 33 bytes
+constexpr uint32_t kPre = 16;       // bytes before a chunk (one needed for the boundary test)
 constexpr uint32_t kSlack = 64;     // gathers read up to 48 bytes past a token start
-constexpr uint32_t kCountSlots = 2048;
 constexpr uint32_t kListRead = 65536;  // list file gread granularity
 constexpr uint32_t kListChunk = 4096;  // list parse granularity (one block per chunk)
 constexpr uint64_t kPairEmpty = ~0ull;
 constexpr uint64_t kDupBit = 1ull << 63;  // table entry: the word has duplicates
+constexpr uint64_t kKeepMagic = 0x31504545504b5247ull;  // GRKPEEP1: the persistent words are initialised
+constexpr uint64_t kPairsClean = 0x4e41454c43524150ull;  // PAIRCLEAN: the (file, word) table is empty
+constexpr uint32_t kRecPage = 2048;  // records per output page
+constexpr uint32_t kNoPage = 0xFFFFFFFFu;
+
+// One work item (a whole file, or a chunk of a large one), precomputed by
+// k_grep_items so the scan needs one round trip per item (32 bytes).
+struct ItemDesc {
+  uint64_t roff;    // file offset of the read: chunk start - pre
+  uint32_t f;       // list index
+  int32_t fd;
+  uint32_t gid;     // reported file id
+  uint32_t rlen;    // bytes to read (chunk + halos, clipped at EOF)
+  uint32_t body;    // bytes whose token starts this item counts (the chunk)
+  uint32_t meta;    // bit 31: a whole file (records emitted directly); bits 0..4: pre (bytes before the chunk)
+};
 
 struct GrepWork {
   // dictionary
@@ -67,22 +88,33 @@ struct GrepWork {
   // file list
   uint8_t* list;          // list_cap bytes
   uint32_t* list_chunk;   // per list chunk: line starts (then exclusive prefix)
-  char* paths;            // max_files * kMaxPath
+  uint64_t* line_off;     // per file: offset of its line in the list
+  const uint32_t* file_ids;  // per file: the id used in records, hits and the digest (NULL: the list index)
   int32_t* fd;
   uint64_t* size;
-  uint64_t* item_base;    // max_files + 1
-  uint32_t* item_file;    // item -> file
+  uint64_t* item_base;    // per file: first item (max_files + 1)
+  struct ItemDesc* desc;  // item -> what to read and where it goes (k_grep_items)
   uint64_t max_items;
+  uint32_t chunk;         // item bytes; also the batch size in batch space
   // (file, word) -> count table
-  uint64_t* pair;         // slot i: pair[2i] = (file << 32) | word (or empty), pair[2i+1] = count;
-                          // key and count share one 32-byte sector
+  uint64_t* pair;         // slot i: pair[2i] = (file << 32) | word (or empty), pair[2i+1] = count
   uint64_t pair_mask;
+  // output records, staged in pages: a block reserves a page of kRecPage
+  // records with ONE atomic and fills it privately (a global counter bumped
+  // per record or per warp serialises at one L2 address, ~14 ns each);
+  // k_grep_pack then packs the used part of every page into d_rec
+  uint32_t* rpool;        // pages of kRecPage records, 3 words each
+  uint32_t* page_used;    // records in each reserved page
+  uint64_t* page_base;    // exclusive prefix of page_used (k_grep_pack)
+  uint64_t max_pages;
   // counters
-  unsigned long long* vars;  // see V_*
-  unsigned long long* prof;  // GFS_GREP_PROF=1: per-phase cycles of k_grep_scan thread 0 (else null)
+  unsigned long long* vars;  // see V_*; cleared every run
+  unsigned long long* keep;  // see K_*; persistent across runs (same work buffer)
+  unsigned long long* prof;  // GFS_GREP_PROF=1: per-phase clock cycles of the scan's thread 0 (else null)
 };
 enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS, V_DSUM, V_DXOR, V_NLISTED,
-       V_NEXTF, V_LISTSZ, V_HOLD_DICT, V_HOLD_LIST, V_NVARS };
+       V_NEXTF, V_LISTSZ, V_HOLD_DICT, V_HOLD_LIST, V_NBATCH, V_NPAGES, V_PAIRS_DIRTY, V_NVARS };
+enum { K_MAGIC = 0, K_PAIRS, K_DICT_FD, K_LIST_FD, K_NKEEP };
 
 __device__ __forceinline__ bool is_word(uint32_t ch) {
   return (ch - 'a' < 26u) || (ch - 'A' < 26u) || (ch - '0' < 10u) || ch == '_';
@@ -116,11 +148,17 @@ __device__ __forceinline__ uint32_t word_bits32(const uint8_t* p) {
 // match is confirmed by an exact 32-byte compare, and the table keeps each
 // such word in its own entry (k_grep_dict), so lookups stay exact.
 __device__ __forceinline__ uint64_t tok_hash(uint32_t w0, uint32_t w1, uint32_t L) {
-  uint64_t h = (((uint64_t)w1 << 32) | w0) ^ (0x9E3779B97F4A7C15ull * L);
-  h *= 0xBF58476D1CE4E5B9ull;
-  h ^= h >> 29;
-  h *= 0x94D049BB133111EBull;
-  return h ^ (h >> 32);
+  // 32-bit multiply-xorshift rounds (one IMAD each; a 64-bit multiply is ~4):
+  // the low word picks the bucket, the high word is the 31-bit fingerprint
+  uint32_t a = (w0 ^ (L * 0x9E3779B9u)) * 0x85EBCA6Bu;
+  a ^= a >> 13;
+  uint32_t b = (w1 + a) * 0xC2B2AE35u;
+  b ^= b >> 16;
+  a = (a ^ b) * 0x27D4EB2Fu;
+  a ^= a >> 15;
+  b = (b ^ (a >> 7)) * 0x165667B1u;
+  b ^= b >> 15;
+  return ((uint64_t)b << 32) | a;
 }
 
 // Low `nb` (0..4) bytes of a word.
@@ -147,7 +185,7 @@ __device__ __forceinline__ void gather_token(const uint32_t (&W)[12], uint32_t s
 
 // entry bits 32..62 hold a 31-bit fingerprint, 26..31 the length
 __device__ __forceinline__ uint64_t entry_key(uint64_t h, uint32_t len) {
-  return (((h >> 33) & 0x7FFFFFFFull) << 32) | ((uint64_t)len << 26);
+  return (((h >> 32) & 0x7FFFFFFFull) << 32) | ((uint64_t)len << 26);
 }
 __device__ __forceinline__ uint64_t key_bits(uint64_t e) { return (e & ~kDupBit) >> 26; }
 
@@ -168,30 +206,75 @@ __device__ __forceinline__ uint64_t hit_mix_hf(uint64_t hf, uint64_t off, uint64
   return splitmix64(splitmix64(hf + off) + k);
 }
 
-__device__ __forceinline__ void set_err(GrepWork& w, long long e) { atomicMin((long long*)&w.vars[V_ERR], e); }
+__device__ __forceinline__ void set_err(const GrepWork& w, long long e) { atomicMin((long long*)&w.vars[V_ERR], e); }
+
+__device__ __forceinline__ uint32_t gid_of(const GrepWork& w, uint32_t f) { return w.file_ids ? w.file_ids[f] : f; }
 
 // --------------------------------------------------------------- hold
 // One block opens the dictionary and the list before the blocks that read
-// them and closes them after the run: the many short gopen/gclose pairs of
+// them, and releases them after the run: the many short gopen/gclose pairs of
 // the reading blocks then never drop the count to zero, which would make the
 // next opener re-validate the file with the host (close-to-open).
-__global__ void k_grep_hold(const gfs_ctx* c, const char* dict_path, const char* list_path, GrepWork w, int release) {
+// With keep_open the two stay open until the next run (which opens them
+// again, then drops the previous run's references), like the corpus files.
+__global__ void k_grep_hold(const gfs_ctx* c, const char* dict_path, const char* list_path, const __grid_constant__ GrepWork w, int release,
+                            int keep_open) {
   if (!release) {
     const int a = gopen(c, dict_path, GFS_O_RDONLY);
     const int b = gopen(c, list_path, GFS_O_RDONLY);
     if (threadIdx.x == 0) {
       w.vars[V_HOLD_DICT] = (unsigned long long)(long long)a;
       w.vars[V_HOLD_LIST] = (unsigned long long)(long long)b;
+      if (w.keep[K_MAGIC] != kKeepMagic) {  // first run on this work buffer
+        w.keep[K_PAIRS] = 0;
+        w.keep[K_DICT_FD] = (unsigned long long)-1ll;
+        w.keep[K_LIST_FD] = (unsigned long long)-1ll;
+        w.keep[K_MAGIC] = kKeepMagic;
+      }
+      w.vars[V_PAIRS_DIRTY] = w.keep[K_PAIRS] != kPairsClean;
+      w.keep[K_PAIRS] = 0;  // dirty until this run's compact has emptied it again
     }
   } else {
     const int a = (int)(long long)w.vars[V_HOLD_DICT], b = (int)(long long)w.vars[V_HOLD_LIST];
-    if (a >= 0) gclose(c, a);
-    if (b >= 0) gclose(c, b);
+    int ra = a, rb = b;  // references to drop now
+    if (keep_open) {
+      ra = (int)(long long)w.keep[K_DICT_FD];
+      rb = (int)(long long)w.keep[K_LIST_FD];
+    }
+    if (ra >= 0) gclose(c, ra);
+    if (rb >= 0) gclose(c, rb);
+    if (threadIdx.x == 0) {
+      w.keep[K_DICT_FD] = keep_open ? (unsigned long long)(long long)a : (unsigned long long)-1ll;
+      w.keep[K_LIST_FD] = keep_open ? (unsigned long long)(long long)b : (unsigned long long)-1ll;
+    }
+  }
+}
+
+// --------------------------------------------------------------- init
+__global__ void k_grep_init(const __grid_constant__ GrepWork w, uint32_t max_words) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
+  for (uint64_t i = t; i <= w.table_mask; i += stride) w.table[i] = 0;
+  for (uint64_t i = t; i < max_words; i += stride) {
+    w.dup_head[i] = 0;
+    w.dup_next[i] = 0;
+  }
+  if (t < V_NVARS) w.vars[t] = 0;
+}
+
+// The (file, word) table is emptied by every successful run's compact; only
+// a fresh work buffer or a failed run leaves it dirty.
+__global__ void k_grep_pairclear(const __grid_constant__ GrepWork w) {
+  if (!w.vars[V_PAIRS_DIRTY]) return;
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i <= w.pair_mask; i += stride) {
+    w.pair[2 * i] = kPairEmpty;
+    w.pair[2 * i + 1] = 0;
   }
 }
 
 // --------------------------------------------------------------- dictionary
-__global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w, uint32_t max_words) {
+__global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, const __grid_constant__ GrepWork w, uint32_t max_words) {
   const int tid = threadIdx.x;
   const int fd = gopen(c, dict_path, GFS_O_RDONLY);
   if (fd < 0) {
@@ -217,21 +300,28 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
     } else {
       for (uint32_t k = k0 + tid; k < k1; k += blockDim.x) {
         uint8_t* s = w.dict + (size_t)k * 32;
+        uint4 q0 = *(const uint4*)s, q1 = *(const uint4*)(s + 16);
+        uint8_t b[32];
+        memcpy(b, &q0, 16);
+        memcpy(b + 16, &q1, 16);
         uint32_t n = 0;
-        while (n < 32 && s[n]) ++n;
+        while (n < 32 && b[n]) ++n;
         bool ok = n > 0;
-        for (uint32_t i = 0; i < n; ++i) ok &= is_word(s[i]);
+        for (uint32_t i = 0; i < n; ++i) ok &= is_word(b[i]);
         if (!ok) {  // empty slot or non-word byte (R13)
           set_err(w, -EINVAL);
           continue;
         }
         // zero the bytes after the word: the slot becomes the word's padded form
-        // (other threads only ever read bytes [0, n) of a slot of length n)
-        for (uint32_t i = n; i < 32; ++i) s[i] = 0;
-        const uint64_t h = tok_hash(((const uint32_t*)s)[0], ((const uint32_t*)s)[1], n);
+        for (uint32_t i = n; i < 32; ++i) b[i] = 0;
+        memcpy(&q0, b, 16);
+        memcpy(&q1, b + 16, 16);
+        *(uint4*)s = q0;
+        *(uint4*)(s + 16) = q1;
+        const uint64_t h = tok_hash(q0.x, q0.y, n);
         const uint64_t ent = entry_key(h, n) | (k + 1);
         // linear probing from the start of the hash's 4-entry (32-byte) bucket:
-        // lookups read a whole bucket per step (scan_token)
+        // lookups read a whole bucket per step (probe_bucket)
         uint32_t slot = (uint32_t)h & w.table_mask & ~3u;
         for (uint32_t probe = 0; probe <= w.table_mask; ++probe, slot = (slot + 1) & w.table_mask) {
           unsigned long long cur = atomicCAS((unsigned long long*)&w.table[slot], 0ull, (unsigned long long)ent);
@@ -240,7 +330,7 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
             const uint32_t kp = (uint32_t)(cur & ((1u << 26) - 1)) - 1;
             const uint8_t* t = w.dict + (size_t)kp * 32;
             bool same = true;
-            for (uint32_t i = 0; i < n; ++i) same &= t[i] == s[i];
+            for (uint32_t i = 0; i < n; ++i) same &= t[i] == b[i];
             if (same) {  // duplicate dictionary word: chain it behind kp, flag the entry
               w.dup_next[k] = atomicExch(&w.dup_head[kp], k + 1);
               atomicOr((unsigned long long*)&w.table[slot], (unsigned long long)kDupBit);
@@ -256,7 +346,7 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, GrepWork w,
 
 // --------------------------------------------------------------- file list
 // Pass 1: every block greads its 64 KiB pieces of the list file.
-__global__ void k_grep_list_read(const gfs_ctx* c, const char* list_path, GrepWork w, uint64_t list_cap) {
+__global__ void k_grep_list_read(const gfs_ctx* c, const char* list_path, const __grid_constant__ GrepWork w, uint64_t list_cap) {
   const int fd = gopen(c, list_path, GFS_O_RDONLY);
   if (fd < 0) {
     if (threadIdx.x == 0 && blockIdx.x == 0) set_err(w, fd);
@@ -281,41 +371,59 @@ __device__ __forceinline__ bool line_start(const uint8_t* L, uint64_t i) {
 }
 
 // Pass 2: line starts (non-empty lines) per chunk.
-__global__ void k_grep_list_count(GrepWork w) {
-  __shared__ uint32_t cnt_s;
+__global__ void k_grep_list_count(const __grid_constant__ GrepWork w) {
   const uint64_t size = w.vars[V_LISTSZ];
   const uint64_t nch = (size + kListChunk - 1) / kListChunk;
   for (uint64_t ch = blockIdx.x; ch < nch; ch += gridDim.x) {
-    if (threadIdx.x == 0) cnt_s = 0;
-    __syncthreads();
     const uint64_t a = ch * kListChunk, b = min(size, a + kListChunk);
     uint32_t n = 0;
     for (uint64_t i = a + threadIdx.x; i < b; i += blockDim.x) n += line_start(w.list, i);
-    atomicAdd(&cnt_s, n);
+    const uint32_t tot = __reduce_add_sync(0xFFFFFFFFu, n);
+    __shared__ uint32_t wsum[32];
+    if ((threadIdx.x & 31) == 0) wsum[threadIdx.x >> 5] = tot;
     __syncthreads();
-    if (threadIdx.x == 0) w.list_chunk[ch] = cnt_s;
+    if (threadIdx.x == 0) {
+      uint32_t t = 0;
+      for (uint32_t q = 0; q < (blockDim.x + 31) / 32; ++q) t += wsum[q];
+      w.list_chunk[ch] = t;
+    }
     __syncthreads();
   }
 }
 
 // Pass 3 (one block): exclusive scan of the chunk counts.
-__global__ void k_grep_list_scan(GrepWork w, uint32_t max_files) {
-  if (threadIdx.x != 0) return;
+__global__ void k_grep_list_scan(const __grid_constant__ GrepWork w, uint32_t max_files) {
+  __shared__ uint32_t part[1024];
   const uint64_t size = w.vars[V_LISTSZ];
-  const uint64_t nch = (size + kListChunk - 1) / kListChunk;
-  uint32_t run = 0;
-  for (uint64_t ch = 0; ch < nch; ++ch) {
-    const uint32_t v = w.list_chunk[ch];
-    w.list_chunk[ch] = run;
+  const uint32_t nch = (uint32_t)((size + kListChunk - 1) / kListChunk);
+  const uint32_t tid = threadIdx.x, nthr = blockDim.x;
+  const uint32_t per = (nch + nthr - 1) / nthr;
+  const uint32_t a = min(nch, tid * per), b = min(nch, a + per);
+  uint32_t s = 0;
+  for (uint32_t i = a; i < b; ++i) s += w.list_chunk[i];
+  part[tid] = s;
+  __syncthreads();
+  if (tid == 0) {
+    uint32_t run = 0;
+    for (uint32_t q = 0; q < nthr; ++q) {
+      const uint32_t v = part[q];
+      part[q] = run;
+      run += v;
+    }
+    if (run > max_files) set_err(w, -ENOSPC);
+    w.vars[V_NFILES] = run < max_files ? run : max_files;
+  }
+  __syncthreads();
+  uint32_t run = part[tid];
+  for (uint32_t i = a; i < b; ++i) {
+    const uint32_t v = w.list_chunk[i];
+    w.list_chunk[i] = run;
     run += v;
   }
-  if (run > max_files) set_err(w, -ENOSPC);
-  w.vars[V_NFILES] = run < max_files ? run : max_files;
 }
 
-// Pass 4: each line start writes its absolute path (relative paths resolve
-// against the list file's directory, R15).
-__global__ void k_grep_list_emit(GrepWork w, const char* dir, uint32_t dir_len, uint32_t max_files) {
+// Pass 4: the offset of every line (file index = rank among non-empty lines).
+__global__ void k_grep_list_emit(const __grid_constant__ GrepWork w, uint32_t max_files) {
   __shared__ uint32_t warp_tot[32];
   __shared__ uint32_t base_s;
   const uint64_t size = w.vars[V_LISTSZ];
@@ -335,22 +443,7 @@ __global__ void k_grep_list_emit(GrepWork w, const char* dir, uint32_t dir_len, 
       uint32_t k = base_s;
       for (int q = 0; q < wid; ++q) k += warp_tot[q];
       k += __popc(bal & ((1u << lane) - 1));
-      if (start && k < max_files) {
-        uint32_t n = 0;
-        while (i + n < size && L[i + n] != '\n') ++n;
-        char* dst = w.paths + (size_t)k * kMaxPath;
-        uint32_t o = 0;
-        if (L[i] != '/') {
-          for (uint32_t q = 0; q < dir_len && o < kMaxPath - 1; ++q) dst[o++] = dir[q];
-          if (o < kMaxPath - 1) dst[o++] = '/';
-        }
-        if (o + n >= kMaxPath) {
-          set_err(w, -ENAMETOOLONG);
-          n = 0;
-        }
-        for (uint32_t q = 0; q < n; ++q) dst[o + q] = (char)L[i + q];
-        dst[o + n] = 0;
-      }
+      if (start && k < max_files) w.line_off[k] = i;
       __syncthreads();
       if (tid == 0) {
         uint32_t tot = 0;
@@ -363,19 +456,57 @@ __global__ void k_grep_list_emit(GrepWork w, const char* dir, uint32_t dir_len, 
 }
 
 // --------------------------------------------------------------- open files
-__global__ void k_grep_open(const gfs_ctx* c, GrepWork w, uint32_t chunk) {
+// One warp per file: the path is the list line (relative lines are resolved
+// against the list's directory, R15), assembled in shared memory,
+// then gopen + gfstat. Records the file's item count and batch-space weight.
+__device__ __forceinline__ uint64_t item_count(uint64_t size, uint32_t chunk) { return (size + chunk - 1) / chunk; }
+__global__ void __launch_bounds__(32) k_grep_open(const gfs_ctx* c, const __grid_constant__ GrepWork w, const char* dir, uint32_t dir_len,
+                                                  uint32_t max_files) {
+  __shared__ __align__(16) char pbuf[kMaxPath + 32];
   __shared__ uint32_t f_s;
-  const int tid = threadIdx.x;
+  const int lane = threadIdx.x;
   const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
+  const uint64_t lsize = w.vars[V_LISTSZ];
   for (;;) {
-    if (tid == 0) f_s = (uint32_t)atomicAdd(&w.vars[V_NEXTF], 1ull);
-    __syncthreads();
+    if (lane == 0) f_s = (uint32_t)atomicAdd(&w.vars[V_NEXTF], 1ull);
+    __syncwarp();
     const uint32_t f = f_s;
     if (f >= nfiles) break;
-    // first gopen of a file goes to the host; page 0 comes back with it
-    const int fd = gopen(c, w.paths + (size_t)f * kMaxPath, GFS_O_RDONLY | GFS_O_PREFETCH);
+    // assemble the path: [dir '/'] line
+    const uint64_t lo = w.line_off[f];
+    const bool rel = w.list[lo] != '/';
+    uint32_t o = 0;
+    if (rel) {
+      for (uint32_t q = lane; q < dir_len; q += 32) pbuf[q] = dir[q];
+      if (lane == 0) pbuf[dir_len] = '/';
+      o = dir_len + 1;
+    }
+    uint32_t n = 0;  // line length
+    bool toolong = false;
+    for (uint64_t base = lo;; base += 32) {
+      const uint64_t i = base + lane;
+      const uint8_t ch = i < lsize ? w.list[i] : (uint8_t)'\n';
+      const uint32_t nl = __ballot_sync(0xFFFFFFFFu, ch == '\n');
+      const uint32_t lim = nl ? (uint32_t)(__ffs(nl) - 1) : 32u;
+      const uint32_t pos = o + (uint32_t)(base - lo) + lane;
+      if ((uint32_t)lane < lim && pos < kMaxPath) pbuf[pos] = (char)ch;
+      if (nl) {
+        n = (uint32_t)(base - lo) + lim;
+        break;
+      }
+      if (o + (uint32_t)(base - lo) + 32 >= kMaxPath) {
+        toolong = true;
+        break;
+      }
+    }
+    if (o + n >= kMaxPath) toolong = true;
+    if (lane == 0 && !toolong) pbuf[o + n] = 0;
+    __syncwarp();
+    int fd = -ENAMETOOLONG;
+    if (!toolong) fd = gopen(c, pbuf, GFS_O_RDONLY | GFS_O_PREFETCH);  // first gopen: page 0 with the reply
+    else if (lane == 0) set_err(w, -ENAMETOOLONG);
     const int64_t sz = fd >= 0 ? gfstat_size(c, fd) : fd;
-    if (tid == 0) {
+    if (lane == 0) {
       w.fd[f] = fd;
       if (sz < 0) {
         set_err(w, sz);
@@ -383,64 +514,118 @@ __global__ void k_grep_open(const gfs_ctx* c, GrepWork w, uint32_t chunk) {
         w.item_base[f] = 0;
       } else {
         w.size[f] = (uint64_t)sz;
-        w.item_base[f] = ((uint64_t)sz + chunk - 1) / chunk;  // item count; scanned later
+        w.item_base[f] = item_count((uint64_t)sz, w.chunk);  // counts; scanned by k_grep_plan
         atomicAdd(&w.vars[V_BYTES], (unsigned long long)sz);
       }
     }
+    __syncwarp();
+  }
+}
+
+// --------------------------------------------------------------- plan
+// One block: exclusive scan of the per-file item counts (item_base), in
+// tiles of 4 * blockDim counts (each thread 4 consecutive ones), the tile's
+// loads issued before the previous tile's scan is used.
+__global__ void k_grep_plan(const __grid_constant__ GrepWork w) {
+  __shared__ uint64_t wsum[32];
+  __shared__ uint64_t carry_s;
+  const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31, wid = tid >> 5, nw = nthr >> 5;
+  const uint64_t n = w.vars[V_NFILES];
+  const uint64_t tile = 4ull * nthr;
+  if (tid == 0) carry_s = 0;
+  __syncthreads();
+  for (uint64_t t0 = 0; t0 < n; t0 += tile) {
+    uint64_t v[4];
+    uint64_t mine = 0;
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      const uint64_t i = t0 + 4ull * tid + q;
+      v[q] = i < n ? w.item_base[i] : 0;
+      mine += v[q];
+    }
+    uint64_t incl = mine;
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint64_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+      if (lane >= o) incl += t;
+    }
+    if (lane == 31) wsum[wid] = incl;
+    __syncthreads();
+    uint64_t base = carry_s + incl - mine, all = 0;
+    for (int q = 0; q < nw; ++q) {
+      base += q < wid ? wsum[q] : 0;
+      all += wsum[q];
+    }
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      const uint64_t i = t0 + 4ull * tid + q;
+      if (i < n) w.item_base[i] = base;
+      base += v[q];
+    }
+    __syncthreads();
+    if (tid == 0) carry_s += all;
     __syncthreads();
   }
-}
-
-// exclusive scan of item counts -> item_base, one block
-__global__ void k_grep_plan(GrepWork w) {
-  __shared__ uint64_t part[1024];
-  const int tid = threadIdx.x, nthr = blockDim.x;
-  const uint32_t n = (uint32_t)w.vars[V_NFILES];
-  const uint32_t per = (n + nthr - 1) / nthr;
-  const uint32_t a = tid * per, b = min(n, a + per);
-  uint64_t s = 0;
-  for (uint32_t i = a; i < b; ++i) s += w.item_base[i];
-  part[tid] = s;
-  __syncthreads();
   if (tid == 0) {
-    uint64_t run = 0;
-    for (int q = 0; q < nthr; ++q) {
-      const uint64_t v = part[q];
-      part[q] = run;
-      run += v;
-    }
-    if (run > w.max_items) {
+    uint64_t r0 = carry_s;
+    if (r0 > w.max_items) {
       set_err(w, -ENOSPC);
-      run = w.max_items;
+      r0 = w.max_items;
     }
-    w.vars[V_NITEMS] = run;
-    w.item_base[n] = run;
-  }
-  __syncthreads();
-  uint64_t run = part[tid];
-  for (uint32_t i = a; i < b; ++i) {
-    const uint64_t v = w.item_base[i];
-    w.item_base[i] = run;
-    run += v;
+    w.vars[V_NITEMS] = r0;
+    w.item_base[n] = r0;
   }
 }
 
-// item -> file map (one thread per file)
-__global__ void k_grep_items(GrepWork w) {
+// item -> descriptor (file, batch-space offset, what to read)
+__global__ void k_grep_items(const __grid_constant__ GrepWork w) {
   const uint32_t n = (uint32_t)w.vars[V_NFILES];
-  for (uint32_t f = blockIdx.x * blockDim.x + threadIdx.x; f < n; f += gridDim.x * blockDim.x) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
+  for (uint64_t f = t; f < n; f += stride) {
     const uint64_t a = w.item_base[f], b = min(w.item_base[f + 1], w.max_items);
-    for (uint64_t i = a; i < b; ++i) w.item_file[i] = f;
+    const uint64_t size = w.size[f];
+    const uint32_t gid = gid_of(w, (uint32_t)f);
+    const int32_t fd = w.fd[f];
+    for (uint64_t i = a; i < b; ++i) {
+      ItemDesc d;
+      d.f = (uint32_t)f;
+      d.fd = fd;
+      d.gid = gid;
+      if (b - a == 1) {  // a whole file
+        d.roff = 0;
+        d.rlen = (uint32_t)size;
+        d.body = (uint32_t)size;
+        d.meta = 1u << 31;
+      } else {  // chunk [s, e) with up to kPre bytes before and kHalo after
+        const uint64_t s = (i - a) * w.chunk, e = min(size, s + w.chunk);
+        const uint64_t ws = s >= kPre ? s - kPre : 0, we = min(size, e + kHalo);
+        d.roff = ws;
+        d.rlen = (uint32_t)(we - ws);
+        d.body = (uint32_t)(e - s);
+        d.meta = (uint32_t)(s - ws);
+      }
+      w.desc[i] = d;
+    }
   }
 }
 
 // --------------------------------------------------------------- scan
-__device__ __forceinline__ void pair_add(GrepWork& w, uint32_t f, uint32_t k, uint64_t cnt) {
+// Bits [lo, hi) of a 32-bit mask (lo, hi clamped to [0, 32]).
+__device__ __forceinline__ uint32_t bit_range(int lo, int hi) {
+  lo = min(max(lo, 0), 32);
+  hi = min(max(hi, 0), 32);
+  if (hi <= lo) return 0u;
+  const uint32_t upto_hi = hi == 32 ? 0xFFFFFFFFu : ((1u << hi) - 1u);
+  const uint32_t below_lo = lo == 32 ? 0xFFFFFFFFu : ((1u << lo) - 1u);
+  return upto_hi & ~below_lo;
+}
+
+__device__ __noinline__ void pair_add(const GrepWork& w, uint32_t f, uint32_t k, uint64_t cnt) {
   const uint64_t key = ((uint64_t)f << 32) | k;
   uint64_t slot = splitmix64(key) & w.pair_mask;
   for (uint64_t probe = 0; probe <= w.pair_mask; ++probe, slot = (slot + 1) & w.pair_mask) {
-    unsigned long long cur = atomicCAS((unsigned long long*)&w.pair[2 * slot], (unsigned long long)kPairEmpty,
-                                       (unsigned long long)key);
+    const unsigned long long cur = atomicCAS((unsigned long long*)&w.pair[2 * slot], (unsigned long long)kPairEmpty,
+                                             (unsigned long long)key);
     if (cur == kPairEmpty || cur == key) {
       atomicAdd((unsigned long long*)&w.pair[2 * slot + 1], (unsigned long long)cnt);
       return;
@@ -449,10 +634,34 @@ __device__ __forceinline__ void pair_add(GrepWork& w, uint32_t f, uint32_t k, ui
   set_err(w, -ENOSPC);
 }
 
+// Space for n <= kRecPage records in the calling block's current output page
+// (a new page when it does not fit); run by one thread, page state in shared
+// memory. Returns the pool index of the first record, or ~0 when out of pages.
+__device__ uint64_t rec_reserve(const GrepWork& w, uint32_t n, uint32_t* page_s, uint32_t* used_s) {
+  if (*page_s == kNoPage || *used_s + n > kRecPage) {
+    if (*page_s != kNoPage) w.page_used[*page_s] = *used_s;
+    const unsigned long long p = atomicAdd(&w.vars[V_NPAGES], 1ull);
+    if (p >= w.max_pages) {
+      set_err(w, -ENOSPC);
+      *page_s = kNoPage;
+      return ~0ull;
+    }
+    *page_s = (uint32_t)p;
+    *used_s = 0;
+  }
+  const uint64_t base = (uint64_t)*page_s * kRecPage + *used_s;
+  *used_s += n;
+  return base;
+}
+__device__ __forceinline__ void rec_close(const GrepWork& w, uint32_t page, uint32_t used) {
+  if (page != kNoPage) w.page_used[page] = used;
+}
+
 struct ScanAcc {
   uint64_t dsum, dxor, nh;
 };
 
+constexpr uint32_t kCountSlots = 2048;
 // Shared-memory state of one scan block (dynamic shared memory, see scan_smem).
 struct ScanSmem {
   uint8_t* buf;     // kPre + chunk + kHalo + kSlack bytes; file byte p at buf[kPre + p - s]
@@ -466,39 +675,63 @@ struct ScanSmem {
 
 // One hit of word k at file position pos: per-item shared count (spilling to
 // the global table when the probe run is exhausted), digest, optional hit list.
-__device__ __forceinline__ void count_hit(GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
+// shared-memory atomics by address space (a generic atomic on a shared
+// address is slower than ATOMS)
+__device__ __forceinline__ uint32_t atoms_cas(uint32_t* p, uint32_t cmp, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.shared.cas.b32 %0, [%1], %2, %3;" : "=r"(r) : "r"(detail::smem_u32(p)), "r"(cmp), "r"(v)
+               : "memory");
+  return r;
+}
+__device__ __forceinline__ uint32_t atoms_add(uint32_t* p, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.shared.add.u32 %0, [%1], %2;" : "=r"(r) : "r"(detail::smem_u32(p)), "r"(v) : "memory");
+  return r;
+}
+__device__ __forceinline__ void reds_add(uint32_t* p, uint32_t v) {
+  asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(detail::smem_u32(p)), "r"(v) : "memory");
+}
+
+// The rare per-hit paths, out of line (the token loop keeps its registers).
+__device__ __noinline__ void hit_spill(const GrepWork& w, uint32_t f, uint32_t k, uint32_t* spilled) {
+  pair_add(w, f, k, 1);  // this item's records then all go through the global table
+  *spilled = 1;
+}
+__device__ __noinline__ void hit_list(const GrepWork& w, uint32_t f, uint32_t k, uint64_t pos, uint64_t* hits,
+                                      uint64_t hit_cap) {
+  const unsigned long long idx = atomicAdd(&w.vars[V_NLISTED], 1ull);
+  if (idx < hit_cap) {
+    hits[2 * idx] = ((uint64_t)f << 32) | k;
+    hits[2 * idx + 1] = pos;
+  }
+}
+
+// One hit of word k at file position pos: per-item shared count (spilling to
+// the global table when the probe run is exhausted), digest, optional hit list.
+__device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
                                           uint32_t f, uint32_t k, uint64_t pos, uint64_t* hits, uint64_t hit_cap,
                                           ScanAcc& acc) {
   uint32_t cs = (k * 2654435761u) & S.cmask;
   bool done = false;
   for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & S.cmask) {
-    const uint32_t prev = atomicCAS(&S.ckey[cs], 0u, k + 1);
-    if (prev == 0) S.olist[atomicAdd(nocc, 1u)] = (uint16_t)cs;
+    const uint32_t prev = atoms_cas(&S.ckey[cs], 0u, k + 1);
+    if (prev == 0) S.olist[atoms_add(nocc, 1u)] = (uint16_t)cs;
     if (prev == 0 || prev == k + 1) {
-      atomicAdd(&S.ccnt[cs], 1u);
+      reds_add(&S.ccnt[cs], 1u);
       done = true;
       break;
     }
   }
-  if (!done) {  // this item's records then all go through the global table
-    pair_add(w, f, k, 1);
-    *spilled = 1;
-  }
+  if (!done) hit_spill(w, f, k, spilled);
   const uint64_t m = hit_mix_hf(S.hf, pos, k);
   acc.dsum += m;
   acc.dxor ^= m;
   ++acc.nh;
-  if (hits) {
-    const unsigned long long idx = atomicAdd(&w.vars[V_NLISTED], 1ull);
-    if (idx < hit_cap) {
-      hits[2 * idx] = ((uint64_t)f << 32) | k;
-      hits[2 * idx + 1] = pos;
-    }
-  }
+  if (hits) hit_list(w, f, k, pos, hits, hit_cap);
 }
 
 // One token: bytes buf[i, i + L), file position pos, 1 <= L <= 32.
-__device__ __forceinline__ void scan_token(GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
+__device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
                                            uint32_t f, uint32_t i, uint32_t L, uint64_t pos, uint64_t* hits,
                                            uint64_t hit_cap, ScanAcc& acc) {
   // first 8 bytes: three aligned words and two funnel shifts
@@ -556,16 +789,8 @@ __device__ __forceinline__ void scan_token(GrepWork& w, const ScanSmem& S, uint3
 }
 
 // Bits [lo, hi) of a 32-bit mask (lo, hi clamped to [0, 32]).
-__device__ __forceinline__ uint32_t bit_range(int lo, int hi) {
-  lo = min(max(lo, 0), 32);
-  hi = min(max(hi, 0), 32);
-  if (hi <= lo) return 0u;
-  const uint32_t upto_hi = hi == 32 ? 0xFFFFFFFFu : ((1u << hi) - 1u);
-  const uint32_t below_lo = lo == 32 ? 0xFFFFFFFFu : ((1u << lo) - 1u);
-  return upto_hi & ~below_lo;
-}
 
-__global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork w, uint32_t chunk, uint64_t* hits,
+__global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __grid_constant__ GrepWork w, uint32_t chunk, uint64_t* hits,
                                                    uint64_t hit_cap, uint64_t* totals, uint32_t* rec,
                                                    uint64_t rec_cap) {
   extern __shared__ __align__(16) uint8_t sm[];
@@ -581,7 +806,8 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
   S.cmask = kCountSlots - 1;
   uint16_t* tok = S.olist + kCountSlots;  // token starts of one round: <= 32 per thread
   const uint32_t round_stripes = 2u * (uint32_t)nthr;
-  __shared__ uint64_t nxt_item, nxt_size, nxt_base;
+  __shared__ uint64_t nxt_item, nxt_size, nxt_base, nxt_roff;
+  __shared__ uint32_t nxt_body, page_s, used_s;
   __shared__ uint32_t nxt_f;
   __shared__ int32_t nxt_fd;
   __shared__ uint32_t nocc_s, spilled_s;
@@ -595,18 +821,24 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
     const uint64_t it = atomicAdd(&w.vars[V_NEXT], 1ull);
     nxt_item = it;
     if (it < nitems) {
-      const uint32_t f = w.item_file[it];
-      nxt_f = f;
-      nxt_fd = w.fd[f];
-      nxt_size = w.size[f];
-      nxt_base = w.item_base[f];
+      const ItemDesc d = w.desc[it];
+      nxt_f = d.gid;
+      nxt_fd = d.fd;
+      nxt_size = d.rlen;  // whole file: its size
+      nxt_base = (d.meta >> 31) ? ~0ull : d.roff + (d.meta & 31u);  // chunk: its start s
+      nxt_body = d.body;
+      nxt_roff = d.roff;
     }
   };
   for (uint32_t i = tid; i < kCountSlots; i += nthr) {  // dynamic smem is not cleared between launches
     S.ckey[i] = 0;
     S.ccnt[i] = 0;
   }
-  if (tid == 0) prefetch();
+  if (tid == 0) {
+    page_s = kNoPage;
+    used_s = 0;
+    prefetch();
+  }
   long long t_prev = clock64();
   auto lap = [&](int k) {
     if (w.prof && tid == 0) {
@@ -623,18 +855,19 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
     const uint32_t f = nxt_f;
     S.hf = splitmix64(f);
     const int fd = nxt_fd;
-    const uint64_t size = nxt_size;
-    const uint64_t s = (item - nxt_base) * chunk;
+    const bool whole = nxt_base == ~0ull;
+    const uint64_t s = whole ? 0 : nxt_base;
+    const uint64_t e = s + (whole ? nxt_size : nxt_body);
+    const uint64_t ws = nxt_roff;
+    const uint64_t we = ws + nxt_size;  // nxt_size: the read length (rlen)
     if (tid == 0) {
       nocc_s = 0;
       spilled_s = 0;
     }
-    const uint64_t e = min(size, s + chunk);
-    const uint64_t ws = s >= kPre ? s - kPre : 0;
-    const uint64_t we = min(size, e + kHalo);
     // file byte p lands at buf[kPre + p - s]; (dst - ws) % 16 == 0, so gread
     // moves the span with TMA (s is a multiple of the chunk, itself of 16)
     const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
+    // (a lane-parallel gread_lanes by warp 0 measured slower here: 23 % vs 18 % of the item time)
     const int64_t r = gread(c, fd, ws, we - ws, S.buf + vlo);  // starts with a barrier
     lap(1);  // 1: gread
     if (r != (int64_t)(we - ws)) {
@@ -704,8 +937,8 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
     }
     // flush: a whole-file item with no spill owns its records; otherwise merge
     const uint32_t nocc = nocc_s;
-    const bool direct = s == 0 && e == size && !spilled_s && rec;
-    if (direct && tid == 0 && nocc) rbase_s = atomicAdd(&w.vars[V_NREC], (unsigned long long)nocc);
+    const bool direct = whole && !spilled_s && rec;
+    if (direct && tid == 0 && nocc) rbase_s = rec_reserve(w, nocc, &page_s, &used_s);
     __syncthreads();
     if (w.prof && tid == 0) atomicAdd(&w.prof[7], 1ull);  // 7: items
     for (uint32_t q = tid; q < nocc; q += nthr) {
@@ -715,19 +948,18 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
       S.ccnt[cs] = 0;
       if (direct) {
         atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
-        const uint64_t idx = rbase_s + q;
-        if (idx < rec_cap) {
-          rec[3 * idx] = f;
-          rec[3 * idx + 1] = k;
-          rec[3 * idx + 2] = cnt;
-        } else {
-          set_err(w, -ENOSPC);
+        if (rbase_s != ~0ull) {
+          uint32_t* o = w.rpool + 3 * (rbase_s + q);
+          o[0] = f;
+          o[1] = k;
+          o[2] = cnt;
         }
       } else {
         pair_add(w, f, k, cnt);
       }
     }
   }
+  if (tid == 0) rec_close(w, page_s, used_s);
   // block-level digest reduction
   for (int o = 16; o; o >>= 1) {
     acc.dsum += __shfl_xor_sync(0xFFFFFFFFu, acc.dsum, o);
@@ -741,157 +973,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, GrepWork
   }
 }
 
-// ------------------------------------------------------------ warp-item scan
-// The same method as k_grep_scan with one WARP per item (warp-collective
-// gread_warp, the paper's design point P:L256-271): no block barrier in the
-// item loop, so a warp waiting on its lookups or probes never holds up the
-// others. Items are smaller (the chunk, e.g. 8 KiB) so a warp's buffer, mask,
-// count table and token list fit in ~16 KiB of shared memory.
-constexpr uint32_t kWarpSlots = 256;  // per-warp count table (overflow spills to the global table)
-constexpr uint32_t kWarpTok = 2048;   // bytes: 64 stripes x <= 16 token starts x u16
-
-__host__ __device__ __forceinline__ uint32_t warp_region_bytes(uint32_t chunk) {
-  const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
-  const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
-  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + kWarpSlots * 8 + kWarpSlots * 2 + kWarpTok + 16;
-}
-
-__global__ void __launch_bounds__(256) k_grep_scan_warp(const gfs_ctx* c, GrepWork w, uint32_t chunk,
-                                                         uint64_t* hits, uint64_t hit_cap, uint64_t* totals,
-                                                         uint32_t* rec, uint64_t rec_cap) {
-  extern __shared__ __align__(16) uint8_t sm[];
-  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
-  uint8_t* base = sm + (size_t)wid * warp_region_bytes(chunk);
-  const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
-  const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
-  ScanSmem S;
-  S.buf = base;
-  S.mask = (uint32_t*)(base + buf_bytes);
-  S.ckey = S.mask + ((nstripe_max + 1 + 3) & ~3u);
-  S.ccnt = S.ckey + kWarpSlots;
-  S.olist = (uint16_t*)(S.ccnt + kWarpSlots);
-  S.cmask = kWarpSlots - 1;
-  uint16_t* tok = S.olist + kWarpSlots;
-  uint32_t* wv = (uint32_t*)((uint8_t*)tok + kWarpTok);  // [0] occupied slots, [1] spilled
-  const uint64_t nitems = w.vars[V_NITEMS];
-  ScanAcc acc{0, 0, 0};
-  for (uint32_t i = lane; i < kWarpSlots; i += 32) {  // dynamic smem is not cleared between launches
-    S.ckey[i] = 0;
-    S.ccnt[i] = 0;
-  }
-  // lane 0 claims the next item; its fields are loaded by every lane (broadcast)
-  uint64_t item = 0;
-  if (lane == 0) item = atomicAdd(&w.vars[V_NEXT], 1ull);
-  item = __shfl_sync(0xFFFFFFFFu, item, 0);
-  while (item < nitems) {
-    const uint32_t f = w.item_file[item];
-    const int fd = w.fd[f];
-    const uint64_t size = w.size[f];
-    const uint64_t s = (item - w.item_base[f]) * chunk;
-    uint64_t next = 0;  // claimed now, so its fields' loads overlap this item
-    if (lane == 0) {
-      next = atomicAdd(&w.vars[V_NEXT], 1ull);
-      wv[0] = 0;
-      wv[1] = 0;
-    }
-    S.hf = splitmix64(f);
-    const uint64_t e = min(size, s + chunk);
-    const uint64_t ws = s >= kPre ? s - kPre : 0;
-    const uint64_t we = min(size, e + kHalo);
-    const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
-    const int64_t r = gread_warp(c, fd, ws, we - ws, S.buf + vlo);
-    next = __shfl_sync(0xFFFFFFFFu, next, 0);
-    if (r != (int64_t)(we - ws)) {
-      if (lane == 0) set_err(w, r < 0 ? r : -EIO);
-      item = next;
-      continue;
-    }
-    // pass 1: word-byte bits per 32-byte stripe; bytes outside [vlo, vhi) are non-word
-    const uint32_t nstripe = (vhi + 31) / 32;
-    for (uint32_t j = lane; j < nstripe; j += 32)
-      S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
-    if (lane == 0) S.mask[nstripe] = 0;
-    __syncwarp();
-    // pass 2, 64 stripes per round: token starts in [s, e) compacted into tok
-    const uint32_t olo = kPre, ohi = kPre + (uint32_t)(e - s);
-    const uint32_t jlo = olo / 32, jhi = (ohi - 1) / 32;
-    for (uint32_t r0 = jlo; r0 <= jhi; r0 += 64) {
-      uint32_t st[2];
-      uint32_t cnt = 0;
-#pragma unroll
-      for (int q = 0; q < 2; ++q) {
-        const uint32_t j = r0 + 2 * (uint32_t)lane + q;
-        st[q] = 0;
-        if (j <= jhi) {
-          const uint32_t m = S.mask[j];
-          const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
-          st[q] = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
-        }
-        cnt += __popc(st[q]);
-      }
-      uint32_t incl = cnt;
-      for (int o = 1; o < 32; o <<= 1) {
-        const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
-        if (lane >= o) incl += t;
-      }
-      const uint32_t total = __shfl_sync(0xFFFFFFFFu, incl, 31);
-      uint32_t off = incl - cnt;
-#pragma unroll
-      for (int q = 0; q < 2; ++q) {
-        const uint32_t jb = 32 * (r0 + 2 * (uint32_t)lane + q);
-        for (uint32_t x = st[q]; x; x &= x - 1) tok[off++] = (uint16_t)(jb + __ffs(x) - 1);
-      }
-      __syncwarp();
-      for (uint32_t q = lane; q < total; q += 32) {
-        const uint32_t i = tok[q], j = i >> 5, b = i & 31;
-        const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | S.mask[j];
-        const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
-        if (L <= 32)                                   // no dictionary word is longer (R12)
-          scan_token(w, S, &wv[0], &wv[1], f, i, L, s + i - kPre, hits, hit_cap, acc);
-      }
-      __syncwarp();  // tok is reused by the next round
-    }
-    // flush: a whole-file item with no spill owns its records; otherwise merge
-    const uint32_t nocc = wv[0];
-    const bool direct = s == 0 && e == size && !wv[1] && rec;
-    unsigned long long rbase = 0;
-    if (direct && lane == 0 && nocc) rbase = atomicAdd(&w.vars[V_NREC], (unsigned long long)nocc);
-    rbase = __shfl_sync(0xFFFFFFFFu, rbase, 0);
-    for (uint32_t q = lane; q < nocc; q += 32) {
-      const uint32_t cs = S.olist[q];
-      const uint32_t k = S.ckey[cs] - 1, cnt = S.ccnt[cs];
-      S.ckey[cs] = 0;
-      S.ccnt[cs] = 0;
-      if (direct) {
-        atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
-        const uint64_t idx = rbase + q;
-        if (idx < rec_cap) {
-          rec[3 * idx] = f;
-          rec[3 * idx + 1] = k;
-          rec[3 * idx + 2] = cnt;
-        } else {
-          set_err(w, -ENOSPC);
-        }
-      } else {
-        pair_add(w, f, k, cnt);
-      }
-    }
-    __syncwarp();  // count table and wv are reset before the next item uses them
-    item = next;
-  }
-  for (int o = 16; o; o >>= 1) {
-    acc.dsum += __shfl_xor_sync(0xFFFFFFFFu, acc.dsum, o);
-    acc.dxor ^= __shfl_xor_sync(0xFFFFFFFFu, acc.dxor, o);
-    acc.nh += __shfl_xor_sync(0xFFFFFFFFu, acc.nh, o);
-  }
-  if (lane == 0) {
-    atomicAdd(&w.vars[V_DSUM], (unsigned long long)acc.dsum);
-    atomicXor(&w.vars[V_DXOR], (unsigned long long)acc.dxor);
-    atomicAdd(&w.vars[V_NHITS], (unsigned long long)acc.nh);
-  }
-}
-
-__global__ void k_grep_close(const gfs_ctx* c, GrepWork w) {
+__global__ void k_grep_close(const gfs_ctx* c, const __grid_constant__ GrepWork w) {
   const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
   for (uint32_t f = blockIdx.x; f < nfiles; f += gridDim.x) {
     const int fd = w.fd[f];
@@ -899,18 +981,24 @@ __global__ void k_grep_close(const gfs_ctx* c, GrepWork w) {
   }
 }
 
-// Unique records from the (file, word) table + word totals. A block takes
-// 1024 consecutive slots (4 per thread, 64 contiguous bytes), scans the valid
-// counts and reserves its output range with one atomic.
-__global__ void __launch_bounds__(256) k_grep_compact(GrepWork w, uint32_t* rec, uint64_t rec_cap,
+// Records of the (file, word) table (chunked files, spilled items) + their
+// word totals. A block takes 1024 consecutive slots (4 per thread, 64
+// contiguous bytes), reserves output space for the valid ones in its record
+// page, and empties the slots again for the next run.
+__global__ void __launch_bounds__(256) k_grep_compact(const __grid_constant__ GrepWork w, int want_rec,
                                                       uint64_t* totals) {
   __shared__ uint32_t warp_tot[8];
+  __shared__ uint32_t page_s, used_s;
   __shared__ unsigned long long base_s;
   const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
+  if (tid == 0) {
+    page_s = kNoPage;
+    used_s = 0;
+  }
   const uint64_t n = w.pair_mask + 1;  // a power of two >= 1024
   for (uint64_t blk = blockIdx.x; blk * 1024 < n; blk += gridDim.x) {
     const uint64_t i0 = blk * 1024 + (uint64_t)tid * 4;
-    const uint4* src = (const uint4*)(w.pair + 2 * i0);
+    uint4* src = (uint4*)(w.pair + 2 * i0);
     uint64_t key[4], cnt[4];
     uint32_t nv = 0;
 #pragma unroll
@@ -933,7 +1021,7 @@ __global__ void __launch_bounds__(256) k_grep_compact(GrepWork w, uint32_t* rec,
       before += q < wid ? t : 0u;
       all += t;
     }
-    if (tid == 0) base_s = all ? atomicAdd(&w.vars[V_NREC], (unsigned long long)all) : 0ull;
+    if (tid == 0) base_s = (all && want_rec) ? rec_reserve(w, all, &page_s, &used_s) : ~0ull;
     __syncthreads();
     uint64_t idx = base_s + before + incl - nv;
 #pragma unroll
@@ -941,35 +1029,63 @@ __global__ void __launch_bounds__(256) k_grep_compact(GrepWork w, uint32_t* rec,
       if (key[q] == kPairEmpty) continue;
       const uint32_t k = (uint32_t)key[q];
       atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt[q]);
-      if (idx < rec_cap) {
-        rec[3 * idx] = (uint32_t)(key[q] >> 32);
-        rec[3 * idx + 1] = k;
-        rec[3 * idx + 2] = (uint32_t)cnt[q];
-      } else if (rec) {
-        set_err(w, -ENOSPC);
+      if (base_s != ~0ull) {
+        uint32_t* o = w.rpool + 3 * idx;
+        o[0] = (uint32_t)(key[q] >> 32);
+        o[1] = k;
+        o[2] = (uint32_t)cnt[q];
       }
       ++idx;
+      src[q] = make_uint4(0xFFFFFFFFu, 0xFFFFFFFFu, 0u, 0u);  // empty again for the next run
     }
     __syncthreads();  // warp_tot / base_s reuse
   }
+  if (tid == 0) rec_close(w, page_s, used_s);
 }
 
-__global__ void k_grep_init(GrepWork w, uint32_t max_words) {
-  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-  const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
-  for (uint64_t i = t; i <= w.pair_mask; i += stride) {
-    w.pair[2 * i] = kPairEmpty;
-    w.pair[2 * i + 1] = 0;
+// Pack the used part of every record page into d_rec: one block scans the
+// page counts (k_grep_pack_scan), then a grid copies the pages.
+__global__ void k_grep_pack_scan(const __grid_constant__ GrepWork w, uint64_t rec_cap) {
+  __shared__ uint64_t part[1024];
+  const uint32_t tid = threadIdx.x, nthr = blockDim.x;
+  const uint64_t np = min((uint64_t)w.vars[V_NPAGES], w.max_pages);
+  const uint64_t per = (np + nthr - 1) / nthr;
+  const uint64_t a = min(np, tid * per), b = min(np, a + per);
+  uint64_t s = 0;
+  for (uint64_t i = a; i < b; ++i) s += w.page_used[i];
+  part[tid] = s;
+  __syncthreads();
+  if (tid == 0) {
+    uint64_t run = 0;
+    for (uint32_t q = 0; q < nthr; ++q) {
+      const uint64_t v = part[q];
+      part[q] = run;
+      run += v;
+    }
+    w.vars[V_NREC] = run;
+    if (run > rec_cap) set_err(w, -ENOSPC);
   }
-  for (uint64_t i = t; i <= w.table_mask; i += stride) w.table[i] = 0;
-  for (uint64_t i = t; i < max_words; i += stride) {
-    w.dup_head[i] = 0;
-    w.dup_next[i] = 0;
+  __syncthreads();
+  uint64_t run = part[tid];
+  for (uint64_t i = a; i < b; ++i) {
+    w.page_base[i] = run;
+    run += w.page_used[i];
   }
-  if (t < V_NVARS) w.vars[t] = 0;
 }
 
-__global__ void k_grep_summary(GrepWork w, uint64_t* out) {
+__global__ void k_grep_pack_copy(const __grid_constant__ GrepWork w, uint32_t* rec, uint64_t rec_cap) {
+  const uint64_t np = min((uint64_t)w.vars[V_NPAGES], w.max_pages);
+  for (uint64_t p = blockIdx.x; p < np; p += gridDim.x) {
+    const uint64_t base = w.page_base[p];
+    const uint64_t lim = base < rec_cap ? rec_cap - base : 0ull;
+    const uint64_t n = (uint64_t)w.page_used[p] < lim ? (uint64_t)w.page_used[p] : lim;
+    const uint32_t* src = w.rpool + 3 * (p * kRecPage);
+    uint32_t* dst = rec + 3 * base;
+    for (uint64_t i = threadIdx.x; i < 3 * n; i += blockDim.x) dst[i] = src[i];
+  }
+}
+
+__global__ void k_grep_summary(const __grid_constant__ GrepWork w, uint64_t* out) {
   if (threadIdx.x == 0) {
     out[0] = w.vars[V_NREC];
     out[1] = w.vars[V_NHITS];
@@ -981,9 +1097,13 @@ __global__ void k_grep_summary(GrepWork w, uint64_t* out) {
     out[7] = w.vars[V_ERR];
     out[8] = w.vars[V_NLISTED];
     out[9] = w.vars[V_NITEMS];
+    // compact emptied every used slot: the next run skips the full clear
+    if (w.vars[V_ERR] == 0) w.keep[K_PAIRS] = kPairsClean;
   }
 }
 
+// Minimum batch-space weight of a whole-file item: chunk/16 rounded up to a
+// stripe, so segments stay 32-byte aligned and a batch holds <= 17 items.
 uint64_t pow2_at_least(uint64_t x) {
   uint64_t p = 1;
   while (p < x) p <<= 1;
@@ -991,35 +1111,42 @@ uint64_t pow2_at_least(uint64_t x) {
 }
 
 struct Layout {
-  uint64_t off[16];
+  uint64_t off[18];
   uint64_t total;
-  uint64_t max_items;
+  uint64_t max_items, tcap, pcap, max_pages;
 };
 
 Layout layout(const gfs_grep_params* p) {
   Layout L{};
-  const uint64_t tcap = pow2_at_least(p->max_words * 8ull < 1024 ? 1024 : p->max_words * 8ull);
-  const uint64_t pcap = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap);
+  L.tcap = pow2_at_least(p->max_words * 8ull < 1024 ? 1024 : p->max_words * 8ull);
+  L.pcap = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap);
+  const uint64_t chunk = p->chunk ? p->chunk : 1;
   // items: one per chunk of corpus plus one partial chunk per file
-  L.max_items = p->corpus_cap / (p->chunk ? p->chunk : 1) + p->max_files + 1;
+  L.max_items = p->corpus_cap / chunk + p->max_files + 1;
+  // record pages: the records themselves plus one partly used page per block
+  // of the scan (<= 8 per SM) and of compact (4 per SM), 160 SMs at most
+  L.max_pages = p->rec_cap / kRecPage + 160 * 12 + 2;
   const uint64_t sizes[] = {
-      (uint64_t)p->max_words * 32,                         // dict
-      tcap * 8,                                            // table
-      (uint64_t)p->max_words * 4,                          // dup_head
-      (uint64_t)p->max_words * 4,                          // dup_next
-      p->list_cap + 64,                                    // list
-      (p->list_cap / kListChunk + 2) * 4,                  // list_chunk
-      (uint64_t)p->max_files * kMaxPath,                   // paths
-      (uint64_t)p->max_files * 4,                          // fd
-      (uint64_t)p->max_files * 8,                          // size
-      ((uint64_t)p->max_files + 1) * 8,                    // item_base
-      L.max_items * 4,                                     // item_file
-      pcap * 16,                                           // pair
-      0,                                                   // (unused)
-      V_NVARS * 8,                                         // vars
+      (uint64_t)p->max_words * 32,                         // 0 dict
+      L.tcap * 8,                                          // 1 table
+      (uint64_t)p->max_words * 4,                          // 2 dup_head
+      (uint64_t)p->max_words * 4,                          // 3 dup_next
+      p->list_cap + 64,                                    // 4 list
+      (p->list_cap / kListChunk + 2) * 4,                  // 5 list_chunk
+      (uint64_t)p->max_files * 8,                          // 6 line_off
+      (uint64_t)p->max_files * 4,                          // 7 fd
+      (uint64_t)p->max_files * 8,                          // 8 size
+      ((uint64_t)p->max_files + 1) * 8,                    // 9 item_base
+      L.max_items * sizeof(ItemDesc),                      // 10 desc
+      L.pcap * 16,                                         // 11 pair
+      L.max_pages * kRecPage * 12,                         // 12 record pages
+      L.max_pages * 4,                                     // 13 page_used
+      L.max_pages * 8,                                     // 14 page_base
+      V_NVARS * 8,                                         // 15 vars
+      K_NKEEP * 8,                                         // 16 keep (persistent)
   };
   uint64_t o = 0;
-  for (int i = 0; i < 14; ++i) {
+  for (int i = 0; i < 17; ++i) {
     L.off[i] = o;
     o += (sizes[i] + 255) & ~255ull;
   }
@@ -1030,8 +1157,7 @@ Layout layout(const gfs_grep_params* p) {
 uint32_t scan_smem(uint32_t chunk, uint32_t block) {
   const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
   const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
-  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * kCountSlots * 4 + kCountSlots * 2 +
-         64 * block;  // token list: <= 32 starts per thread per round (2 bytes each)
+  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * kCountSlots * 4 + kCountSlots * 2 + 64 * block;
 }
 
 }  // namespace
@@ -1042,7 +1168,8 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
                      const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
                      uint64_t* d_hits, uint64_t* d_summary) {
   if (!h || !dict_path || !list_path || !p || !d_work || !d_totals || !d_summary || p->max_files == 0 ||
-      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) || p->chunk + kPre + kHalo > 65536 ||  // u16 token offsets
+      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) ||
+      p->chunk + kPre + kHalo > 65536 ||  // 16-bit token offsets into the item buffer
       p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31))
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
@@ -1051,134 +1178,96 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   GrepWork w;
   w.dict = base + L.off[0];
   w.table = (uint64_t*)(base + L.off[1]);
-  w.table_mask = (uint32_t)(pow2_at_least(p->max_words * 8ull < 1024 ? 1024 : p->max_words * 8ull) - 1);
+  w.table_mask = (uint32_t)(L.tcap - 1);
   w.dup_head = (uint32_t*)(base + L.off[2]);
   w.dup_next = (uint32_t*)(base + L.off[3]);
   w.list = base + L.off[4];
   w.list_chunk = (uint32_t*)(base + L.off[5]);
-  w.paths = (char*)(base + L.off[6]);
+  w.line_off = (uint64_t*)(base + L.off[6]);
+  w.file_ids = p->file_ids;
   w.fd = (int32_t*)(base + L.off[7]);
   w.size = (uint64_t*)(base + L.off[8]);
   w.item_base = (uint64_t*)(base + L.off[9]);
-  w.item_file = (uint32_t*)(base + L.off[10]);
+  w.desc = (ItemDesc*)(base + L.off[10]);
   w.max_items = L.max_items;
+  w.chunk = p->chunk;
   w.pair = (uint64_t*)(base + L.off[11]);
-  w.pair_mask = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap) - 1;
-  w.vars = (unsigned long long*)(base + L.off[13]);
+  w.pair_mask = L.pcap - 1;
+  w.rpool = (uint32_t*)(base + L.off[12]);
+  w.page_used = (uint32_t*)(base + L.off[13]);
+  w.page_base = (uint64_t*)(base + L.off[14]);
+  w.max_pages = L.max_pages;
+  w.vars = (unsigned long long*)(base + L.off[15]);
+  w.keep = (unsigned long long*)(base + L.off[16]);
 
-  // staged strings: dict path, list path, list directory
-  static char* d_str = nullptr;
-  static char* h_str = nullptr;
-  static cudaEvent_t ev = nullptr;
-  if (!d_str) {
-    if (cudaMalloc((void**)&d_str, 3 * kMaxPath) != cudaSuccess) return -ENOMEM;
-    if (cudaHostAlloc((void**)&h_str, 3 * kMaxPath, cudaHostAllocPortable) != cudaSuccess) return -ENOMEM;
-    cudaEventCreateWithFlags(&ev, cudaEventDisableTiming);
-  } else {
-    cudaEventSynchronize(ev);
+  // path arguments: dictionary, list, the list's directory (relative lines)
+  gfs_launch::ArgStage as(h, s);
+  std::string dir;
+  {
+    const char* slash = strrchr(list_path, '/');
+    dir = slash ? std::string(list_path, (size_t)(slash - list_path)) : std::string(".");
+    if (dir.empty()) dir = "/";  // a list at the root: "/" + "/" + line still resolves
   }
-  const size_t nd = strlen(dict_path), nl = strlen(list_path);
-  if (nd >= kMaxPath || nl >= kMaxPath) return -ENAMETOOLONG;
-  memcpy(h_str, dict_path, nd + 1);
-  memcpy(h_str + kMaxPath, list_path, nl + 1);
-  const char* slash = strrchr(list_path, '/');
-  size_t dl = 0;
-  if (slash) {
-    dl = (size_t)(slash - list_path);
-    memcpy(h_str + 2 * kMaxPath, list_path, dl);
-  } else {
-    h_str[2 * kMaxPath] = '.';
-    dl = 1;
-  }
-  h_str[2 * kMaxPath + dl] = 0;
-  cudaMemcpyAsync(d_str, h_str, 3 * kMaxPath, cudaMemcpyHostToDevice, s);
-  cudaEventRecord(ev, s);
+  const char* strs[3] = {dict_path, list_path, dir.c_str()};
+  if (const int e = as.stage(strs, 3)) return e;
+  const char* d_dict = as.str(0);
+  const char* d_list = as.str(1);
+  const char* d_dir = as.str(2);
 
   const gfs_ctx* c = gfs_device_ctx(h);
-  // GFS_GREP_WARP=1: one warp per item (k_grep_scan_warp)
-  const bool warp_items = getenv("GFS_GREP_WARP") && *getenv("GFS_GREP_WARP") == '1';
-  const uint32_t smem = warp_items ? warp_region_bytes(p->chunk) * (p->block / 32) : scan_smem(p->chunk, p->block);
-  if (smem > 227 * 1024) return -EINVAL;
-  if (warp_items && p->block / 32 > GFS_WARP_API_MAX_WARPS) return -EINVAL;
-  cudaFuncSetAttribute(warp_items ? (const void*)k_grep_scan_warp : (const void*)k_grep_scan,
-                       cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-  // GFS_GREP_DEBUG=1: synchronise after each stage, print its time and the first error
-  const bool dbg = getenv("GFS_GREP_DEBUG") && *getenv("GFS_GREP_DEBUG") == '1';
-  static unsigned long long* d_prof = nullptr;
+  static unsigned long long* d_prof = nullptr;  // GFS_GREP_PROF=1 (diagnostics only)
   w.prof = nullptr;
   if (getenv("GFS_GREP_PROF") && *getenv("GFS_GREP_PROF") == '1') {
     if (!d_prof && cudaMalloc((void**)&d_prof, 8 * sizeof(unsigned long long)) != cudaSuccess) d_prof = nullptr;
     if (d_prof) cudaMemsetAsync(d_prof, 0, 8 * sizeof(unsigned long long), s);
     w.prof = d_prof;
   }
-  struct timespec ts_prev;
-  clock_gettime(CLOCK_MONOTONIC, &ts_prev);
-  auto stage = [&](const char* name) {
-    if (!dbg) return;
-    cudaError_t e = cudaStreamSynchronize(s);
-    struct timespec ts;
-    clock_gettime(CLOCK_MONOTONIC, &ts);
-    unsigned long long v[V_NVARS];
-    cudaMemcpy(v, w.vars, sizeof(v), cudaMemcpyDeviceToHost);
-    fprintf(stderr, "gfs_grep[%s]: %.3f ms cuda=%s err=%lld nfiles=%llu nwords=%llu nitems=%llu bytes=%llu\n", name,
-            (ts.tv_sec - ts_prev.tv_sec) * 1e3 + (ts.tv_nsec - ts_prev.tv_nsec) * 1e-6, cudaGetErrorString(e),
-            (long long)v[V_ERR], v[V_NFILES], v[V_NWORDS], v[V_NITEMS], v[V_BYTES]);
-    ts_prev = ts;
-  };
+  const uint32_t smem = scan_smem(p->chunk, p->block);
+  if (smem > 227 * 1024) return -EINVAL;
+  cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  int dev = 0, nsm = 148;
+  cudaGetDevice(&dev);
+  cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
   const uint64_t lb = p->list_cap / kListChunk + 1, lr = p->list_cap / kListRead + 1;
   const uint32_t list_blocks = (uint32_t)(lb < 1024 ? lb : 1024);
   // one opener per 64 KiB piece: a block that opens the list after all others
   // closed it would re-validate it with the host (close-to-open)
   const uint32_t read_blocks = (uint32_t)(lr < 1024 ? lr : 1024);
-  k_grep_init<<<1024, 256, 0, s>>>(w, p->max_words);
-  k_grep_hold<<<1, 32, 0, s>>>(c, d_str, d_str + kMaxPath, w, 0);
-  k_grep_dict<<<64, 256, 0, s>>>(c, d_str, w, p->max_words);
-  stage("dict");
-  k_grep_list_read<<<read_blocks, 256, 0, s>>>(c, d_str + kMaxPath, w, p->list_cap);
+  k_grep_init<<<nsm * 4, 256, 0, s>>>(w, p->max_words);
+  k_grep_hold<<<1, 32, 0, s>>>(c, d_dict, d_list, w, 0, (int)p->keep_open);
+  k_grep_pairclear<<<nsm * 4, 256, 0, s>>>(w);
+  k_grep_dict<<<nsm, 256, 0, s>>>(c, d_dict, w, p->max_words);
+  k_grep_list_read<<<read_blocks, 256, 0, s>>>(c, d_list, w, p->list_cap);
   k_grep_list_count<<<list_blocks, 256, 0, s>>>(w);
-  k_grep_list_scan<<<1, 32, 0, s>>>(w, p->max_files);
-  k_grep_list_emit<<<list_blocks, 256, 0, s>>>(w, d_str + 2 * kMaxPath, (uint32_t)dl, p->max_files);
-  stage("list");
-  // gopen is block-collective with one leader thread: many one-warp blocks
-  // keep more opens in flight (host RPCs when cold, L2 round trips when warm)
-  int dev = 0, nsm = 148;
-  cudaGetDevice(&dev);
-  cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
-  k_grep_open<<<nsm * 16, 32, 0, s>>>(c, w, p->chunk);
-  stage("open");
+  k_grep_list_scan<<<1, 1024, 0, s>>>(w, p->max_files);
+  k_grep_list_emit<<<list_blocks, 256, 0, s>>>(w, p->max_files);
+  // gopen is collective with one leader thread: many one-warp blocks keep
+  // more opens in flight (host RPCs when cold, L2 round trips when warm)
+  k_grep_open<<<nsm * 32, 32, 0, s>>>(c, w, d_dir, (uint32_t)dir.size(), p->max_files);
   k_grep_plan<<<1, 1024, 0, s>>>(w);
-  k_grep_items<<<256, 256, 0, s>>>(w);
+  k_grep_items<<<nsm * 2, 256, 0, s>>>(w);
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
   // persistent scan grid: every resident block slot once (p->grid caps it)
   int occ = 1;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, warp_items ? (const void*)k_grep_scan_warp
-                                                                 : (const void*)k_grep_scan, (int)p->block, smem);
-  // GFS_GREP_BPS=n: at most n scan blocks per SM, the rest of the SM's
-  // L1/shared-memory array left to L1 (dictionary buckets of frequent words)
-  if (getenv("GFS_GREP_BPS")) {
-    const int cap = atoi(getenv("GFS_GREP_BPS"));
-    if (cap > 0 && cap < occ) occ = cap;
-    const int pct = (int)((occ * (uint64_t)(smem + 1024) * 100 + 228 * 1024 - 1) / (228 * 1024));
-    cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributePreferredSharedMemoryCarveout, pct < 100 ? pct : 100);
-  }
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_scan, (int)p->block, smem);
   const uint32_t scan_grid = (uint32_t)(occ > 0 ? occ : 1) * (uint32_t)nsm;
-  if (warp_items)
-    k_grep_scan_warp<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
-        c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
-  else
-    k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
-        c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
-  stage("scan");
+  k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
+      c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
   if (!p->keep_open) k_grep_close<<<nsm * 16, 32, 0, s>>>(c, w);
-  k_grep_compact<<<nsm * 8, 256, 0, s>>>(w, d_rec, d_rec ? rec_cap : 0, d_totals);
-  k_grep_hold<<<1, 32, 0, s>>>(c, d_str, d_str + kMaxPath, w, 1);
+  k_grep_compact<<<nsm * 4, 256, 0, s>>>(w, d_rec ? 1 : 0, d_totals);
+  if (d_rec) {
+    k_grep_pack_scan<<<1, 1024, 0, s>>>(w, rec_cap);
+    k_grep_pack_copy<<<nsm * 8, 256, 0, s>>>(w, d_rec, rec_cap);
+  }
+  k_grep_hold<<<1, 32, 0, s>>>(c, d_dict, d_list, w, 1, (int)p->keep_open);
   k_grep_summary<<<1, 32, 0, s>>>(w, d_summary);
-  stage("done");
   if (w.prof) {
     unsigned long long pv[8];
     cudaMemcpyAsync(pv, w.prof, sizeof(pv), cudaMemcpyDeviceToHost, s);
     cudaStreamSynchronize(s);
-    const double tot = (double)(pv[0] + pv[1] + pv[2] + pv[3] + pv[4] + pv[5]) + 1e-9;
+    double tot = 0;
+    for (int i = 0; i < 6; ++i) tot += (double)pv[i];
+    tot += 1e-9;
     fprintf(stderr, "gfs_grep[scan prof, thread 0 cycles]: items=%llu loop-top=%.1f%% gread=%.1f%% pass1=%.1f%% "
             "toklist=%.1f%% tokens=%.1f%% wait-others=%.1f%% (%.0f cycles/item)\n", pv[7], 100 * pv[0] / tot,
             100 * pv[1] / tot, 100 * pv[2] / tot, 100 * pv[3] / tot, 100 * pv[4] / tot, 100 * pv[5] / tot,

@@ -47,6 +47,7 @@
 #include <cuda_runtime.h>
 
 #include "gpufs.h"
+#include "gfs_launch.h"
 
 #define GFS_API extern "C" __attribute__((visibility("default")))
 
@@ -254,6 +255,16 @@ struct gfs_handle {
   SpinMutex zc_mu;
   std::vector<ZcFile> zc;
   std::vector<void*> ipc_open;   // CUDA IPC mappings to close at shutdown
+  // Launcher argument staging (path strings for the kernels): a ring of slots
+  // in pinned host + device memory of this handle's device. A slot is reused
+  // only after the event recorded behind the LAST kernel that read it.
+  static constexpr int kArgSlots = 64;
+  char* arg_h = nullptr;
+  char* arg_d = nullptr;
+  cudaEvent_t arg_ev[kArgSlots] = {};
+  bool arg_used[kArgSlots] = {};
+  int arg_next = 0;
+  std::mutex arg_mu;
 };
 
 namespace {
@@ -887,6 +898,10 @@ void free_all(gfs_handle* h) {
   if (h->paths_h) cudaFreeHost(h->paths_h);
   if (h->cpl_h) cudaFreeHost(h->cpl_h);
   if (h->staging_h) cudaFreeHost(h->staging_h);
+  for (int i = 0; i < gfs_handle::kArgSlots; ++i)
+    if (h->arg_ev[i]) cudaEventDestroy(h->arg_ev[i]);
+  F(h->arg_d);
+  if (h->arg_h) cudaFreeHost(h->arg_h);
   if (h->priv) cudaStreamDestroy(h->priv);
   h->vt.close();
 }
@@ -1028,6 +1043,9 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
       goto fail;
     }
   }
+  CK(cudaMalloc((void**)&h->arg_d, (size_t)gfs_handle::kArgSlots * GFS_ARG_SLOT_BYTES));
+  CK(cudaHostAlloc((void**)&h->arg_h, (size_t)gfs_handle::kArgSlots * GFS_ARG_SLOT_BYTES, cudaHostAllocPortable));
+  for (int i = 0; i < gfs_handle::kArgSlots; ++i) CK(cudaEventCreateWithFlags(&h->arg_ev[i], cudaEventDisableTiming));
   CK(cudaMalloc((void**)&h->d, sizeof(gfs_ctx)));
   CK(cudaMemcpyAsync(h->d, &c, sizeof(gfs_ctx), cudaMemcpyHostToDevice, h->priv));
   CK(cudaStreamSynchronize(h->priv));
@@ -1082,6 +1100,38 @@ GFS_API int gfs_shutdown(gfs_handle* h) {
 }
 
 GFS_API const gfs_ctx* gfs_device_ctx(gfs_handle* h) { return h ? h->d : nullptr; }
+
+// Launcher argument staging (gfs_launch.h). The strings go to a slot of this
+// handle's ring (host copy, then an async copy on `s`); the caller records the
+// slot's event with gfs_internal_args_done() after enqueuing the last kernel
+// that reads them, and a slot is rewritten only once that event completed —
+// so concurrent launches on different streams never overwrite each other's
+// arguments, and the device memory belongs to the handle's own device.
+extern "C" int gfs_internal_args(gfs_handle* h, cudaStream_t s, const char* const* strs, int n, char** d_out) {
+  if (!h || n < 0 || n > GFS_ARG_SLOT_BYTES / GFS_MAX_PATH) return -EINVAL;
+  for (int i = 0; i < n; ++i)
+    if (!strs[i] || strlen(strs[i]) >= GFS_MAX_PATH) return -ENAMETOOLONG;
+  std::lock_guard<std::mutex> g(h->arg_mu);
+  const int k = h->arg_next;
+  h->arg_next = (k + 1) % gfs_handle::kArgSlots;
+  if (h->arg_used[k]) cudaEventSynchronize(h->arg_ev[k]);
+  char* hp = h->arg_h + (size_t)k * GFS_ARG_SLOT_BYTES;
+  for (int i = 0; i < n; ++i) memcpy(hp + (size_t)i * GFS_MAX_PATH, strs[i], strlen(strs[i]) + 1);
+  char* dp = h->arg_d + (size_t)k * GFS_ARG_SLOT_BYTES;
+  if (n && cudaMemcpyAsync(dp, hp, (size_t)n * GFS_MAX_PATH, cudaMemcpyHostToDevice, s) != cudaSuccess) return -EIO;
+  h->arg_used[k] = false;
+  *d_out = dp;
+  return k;
+}
+
+extern "C" void gfs_internal_args_done(gfs_handle* h, int slot, cudaStream_t s) {
+  if (!h || slot < 0 || slot >= gfs_handle::kArgSlots) return;
+  std::lock_guard<std::mutex> g(h->arg_mu);
+  cudaEventRecord(h->arg_ev[slot], s);
+  h->arg_used[slot] = true;
+}
+
+extern "C" int gfs_internal_device(gfs_handle* h) { return h ? h->cfg.device : -1; }
 
 // ------------------------------------------------------------------ peer caches (NEXT-1)
 namespace {

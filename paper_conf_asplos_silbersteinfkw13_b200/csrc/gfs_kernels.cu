@@ -15,6 +15,7 @@
 
 #include "gpufs.h"
 #include "gpufs_device.cuh"
+#include "gfs_launch.h"
 
 #define GFS_API extern "C" __attribute__((visibility("default")))
 
@@ -434,43 +435,6 @@ __global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, 
 
 int launch_err(cudaError_t e) { return e == cudaSuccess ? 0 : -EIO; }
 
-// Stage a host path string in device memory, ordered on `s`. The staging
-// buffer is a small per-process ring of pinned+device buffers.
-struct PathStage {
-  char* d = nullptr;
-  char* h = nullptr;
-  cudaEvent_t ev[64];
-  bool used[64];
-  int next = 0;
-  bool init = false;
-};
-PathStage g_ps;
-
-const char* stage_path(const char* path, cudaStream_t s) {
-  if (!path) return nullptr;
-  const size_t n = strlen(path);
-  if (n >= GFS_MAX_PATH) return nullptr;
-  if (!g_ps.init) {
-    if (cudaMalloc((void**)&g_ps.d, 64 * GFS_MAX_PATH) != cudaSuccess) return nullptr;
-    if (cudaHostAlloc((void**)&g_ps.h, 64 * GFS_MAX_PATH, cudaHostAllocPortable) != cudaSuccess) return nullptr;
-    for (int i = 0; i < 64; ++i) {
-      cudaEventCreateWithFlags(&g_ps.ev[i], cudaEventDisableTiming);
-      g_ps.used[i] = false;
-    }
-    g_ps.init = true;
-  }
-  const int k = g_ps.next;
-  g_ps.next = (k + 1) % 64;
-  if (g_ps.used[k]) cudaEventSynchronize(g_ps.ev[k]);
-  memcpy(g_ps.h + (size_t)k * GFS_MAX_PATH, path, n + 1);
-  if (cudaMemcpyAsync(g_ps.d + (size_t)k * GFS_MAX_PATH, g_ps.h + (size_t)k * GFS_MAX_PATH, n + 1,
-                      cudaMemcpyHostToDevice, s) != cudaSuccess)
-    return nullptr;
-  cudaEventRecord(g_ps.ev[k], s);
-  g_ps.used[k] = true;
-  return g_ps.d + (size_t)k * GFS_MAX_PATH;
-}
-
 }  // namespace
 
 extern "C" int gfs_internal_init_metadata(gfs_ctx* hctx, cudaStream_t s) {
@@ -486,8 +450,9 @@ GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mod
   if ((mode & 0xFF) >= 4 && (mode >> 8)) return -EINVAL;  // warp harness: read-only opens
   if ((mode & 0xFF) >= 4 && ((block & 31) || block > 32 * GFS_WARP_API_MAX_WARPS)) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = stage_path(path, s);
-  if (!dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(h, s);
+  if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = as.str(0);
   if (mode >= 4 && mode <= 5) {
     const uint32_t dyn = mode == 5 ? smem_bytes * (block / 32) : 0;
     if (dyn > 200 * 1024) return -EINVAL;
@@ -509,8 +474,9 @@ GFS_API int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint6
                             uint32_t grid, uint32_t block) {
   if (!h || grid == 0 || block == 0 || block > 1024 || chunk == 0 || (chunk & 7) || (file_off & 7)) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = stage_path(path, s);
-  if (!dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(h, s);
+  if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = as.str(0);
   k_seqread<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, file_off, total, chunk, use_mmap, d_scratch, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
@@ -522,8 +488,10 @@ GFS_API int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int 
       chunk > 200 * 1024)
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = raw ? nullptr : stage_path(path, s);
-  if (!raw && !dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(raw ? nullptr : h, s);
+  if (!raw)
+    if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = raw ? nullptr : as.str(0);
   if (chunk > 48 * 1024) cudaFuncSetAttribute(k_randread, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
   k_randread<<<grid, block, chunk, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
                                         d_off, d_sum, d_err);
@@ -537,8 +505,10 @@ GFS_API int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path,
       block / 32 > GFS_WARP_API_MAX_WARPS || chunk == 0 || (chunk & 15) || (uint64_t)chunk * (block / 32) > 200 * 1024)
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = raw ? nullptr : stage_path(path, s);
-  if (!raw && !dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(raw ? nullptr : h, s);
+  if (!raw)
+    if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = raw ? nullptr : as.str(0);
   const uint32_t smem = chunk * (block / 32);
   if (smem > 48 * 1024) cudaFuncSetAttribute(k_randread_warp, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   k_randread_warp<<<grid, block, smem, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk,
@@ -552,8 +522,9 @@ GFS_API int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32
   if (!h || grid == 0 || block == 0 || block > 1024) return -EINVAL;
   if (flags != (int)GFS_O_GWRONCE && flags != (int)GFS_O_RDWR) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = stage_path(path, s);
-  if (!dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(h, s);
+  if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = as.str(0);
   k_gwrite_calls<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, flags);
   return launch_err(cudaGetLastError());
 }
@@ -563,8 +534,9 @@ GFS_API int gfs_run_mmap_write(gfs_handle* h, void* stream, const char* path, ui
                                uint32_t grid, uint32_t block, int do_msync) {
   if (!h || grid == 0 || block == 0 || block > 1024) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = stage_path(path, s);
-  if (!dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(h, s);
+  if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = as.str(0);
   k_mmap_write<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, do_msync);
   return launch_err(cudaGetLastError());
 }
@@ -575,8 +547,9 @@ GFS_API int gfs_run_seqwrite(gfs_handle* h, void* stream, const char* path, uint
   if (!h || !d_src || !d_err || !d_tmp || grid == 0 || block == 0 || block > 1024 || sync_grid == 0 || chunk == 0)
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = stage_path(path, s);
-  if (!dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(h, s);
+  if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = as.str(0);
   const gfs_ctx* c = gfs_device_ctx(h);
   // pin: one open held across the launches, so the writers' gclose never
   // closes the file (a later O_GWRONCE open would start a new incarnation)
@@ -592,8 +565,9 @@ GFS_API int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int fl
                            int64_t* d_ret) {
   if (!h || !d_ret) return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  const char* dp = stage_path(path, s);
-  if (!dp) return -ENAMETOOLONG;
+  gfs_launch::ArgStage as(h, s);
+  if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = as.str(0);
   if (op == 6) {  // parallel gfsync: arg = grid; *d_ret = 0 or the most negative error
     if (arg == 0 || arg > 65535) return -EINVAL;
     cudaMemsetAsync(d_ret, 0, 8, s);

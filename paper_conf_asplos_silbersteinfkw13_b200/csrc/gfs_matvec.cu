@@ -24,6 +24,7 @@
 
 #include "gpufs.h"
 #include "gpufs_device.cuh"
+#include "gfs_launch.h"
 
 #define GFS_API extern "C" __attribute__((visibility("default")))
 
@@ -75,14 +76,15 @@ __device__ __forceinline__ double block_sum(double v, double* red) {
   return s;  // valid in thread 0
 }
 
+// Rows [row0, row0 + nrows) of A; y (file and d_y) holds those rows only.
 __global__ void __launch_bounds__(256) k_mv_rows(const gfs_ctx* c, const char* a_path, const char* y_path,
-                                                  uint64_t rows, uint64_t cols, const float* x, float* y_dev,
-                                                  int64_t* err) {
+                                                  uint64_t row0, uint64_t nrows, uint64_t cols, const float* x,
+                                                  float* y_dev, int64_t* err) {
   extern __shared__ __align__(16) float ys[];  // this block's y slice
   __shared__ double red[32];
   const int tid = threadIdx.x, nthr = blockDim.x;
-  const uint64_t per = (rows + gridDim.x - 1) / gridDim.x;
-  const uint64_t r0 = blockIdx.x * per, r1 = r0 + per < rows ? r0 + per : rows;
+  const uint64_t per = (nrows + gridDim.x - 1) / gridDim.x;
+  const uint64_t r0 = row0 + blockIdx.x * per, r1 = r0 + per < row0 + nrows ? r0 + per : row0 + nrows;
   if (r0 >= r1) return;
   const int fa = gopen(c, a_path, GFS_O_RDONLY);
   if (fa < 0) {
@@ -128,13 +130,13 @@ __global__ void __launch_bounds__(256) k_mv_rows(const gfs_ctx* c, const char* a
   __syncthreads();
   if (!ok) return;
   if (y_dev)
-    for (uint64_t i = tid; i < r1 - r0; i += nthr) y_dev[r0 + i] = ys[i];
+    for (uint64_t i = tid; i < r1 - r0; i += nthr) y_dev[r0 - row0 + i] = ys[i];
   const int fy = gopen(c, y_path, GFS_O_GWRONCE);
   if (fy < 0) {
     if (tid == 0) mv_err(err, fy);
     return;
   }
-  const int64_t w = gwrite(c, fy, r0 * 4, (r1 - r0) * 4, ys);
+  const int64_t w = gwrite(c, fy, (r0 - row0) * 4, (r1 - r0) * 4, ys);
   if (tid == 0 && w != (int64_t)((r1 - r0) * 4)) mv_err(err, w < 0 ? w : -EIO);
   gclose(c, fy);
 }
@@ -153,45 +155,36 @@ __global__ void k_mv_sync(const gfs_ctx* c, const char* y_path, int64_t* err) {
 
 }  // namespace
 
-GFS_API int gfs_matvec(gfs_handle* h, void* stream, const char* a_path, const char* x_path, const char* y_path,
-                       uint64_t rows, uint64_t cols, float* d_x, float* d_y, int64_t* d_err, uint32_t grid,
-                       uint32_t block) {
+GFS_API int gfs_matvec_rows(gfs_handle* h, void* stream, const char* a_path, const char* x_path, const char* y_path,
+                            uint64_t rows, uint64_t cols, uint64_t row0, uint64_t nrows, float* d_x, float* d_y,
+                            int64_t* d_err, uint32_t grid, uint32_t block) {
   if (!h || !a_path || !x_path || !y_path || !d_x || !d_err || rows == 0 || cols == 0 || grid == 0 ||
-      block == 0 || block > 256 || (block & 31))
+      block == 0 || block > 256 || (block & 31) || nrows == 0 || row0 >= rows || nrows > rows - row0)
     return -EINVAL;
-  const uint64_t per = (rows + grid - 1) / grid;
+  const uint64_t per = (nrows + grid - 1) / grid;
   if (per * 4 > 160 * 1024) return -EINVAL;  // y slice must fit in shared memory: use more blocks
   cudaStream_t s = (cudaStream_t)stream;
-  static char* d_str = nullptr;
-  static char* h_str = nullptr;
-  static cudaEvent_t ev = nullptr;
-  if (!d_str) {
-    if (cudaMalloc((void**)&d_str, 3 * GFS_MAX_PATH) != cudaSuccess) return -ENOMEM;
-    if (cudaHostAlloc((void**)&h_str, 3 * GFS_MAX_PATH, cudaHostAllocPortable) != cudaSuccess) return -ENOMEM;
-    cudaEventCreateWithFlags(&ev, cudaEventDisableTiming);
-  } else {
-    cudaEventSynchronize(ev);
-  }
+  gfs_launch::ArgStage as(h, s);
   const char* ps[3] = {a_path, x_path, y_path};
-  for (int i = 0; i < 3; ++i) {
-    const size_t n = strlen(ps[i]);
-    if (n >= GFS_MAX_PATH) return -ENAMETOOLONG;
-    memcpy(h_str + i * GFS_MAX_PATH, ps[i], n + 1);
-  }
-  cudaMemcpyAsync(d_str, h_str, 3 * GFS_MAX_PATH, cudaMemcpyHostToDevice, s);
-  cudaEventRecord(ev, s);
+  if (const int e = as.stage(ps, 3)) return e;
   const gfs_ctx* c = gfs_device_ctx(h);
-  const char* da = d_str;
-  const char* dx = d_str + GFS_MAX_PATH;
-  const char* dy = d_str + 2 * GFS_MAX_PATH;
+  const char* da = as.str(0);
+  const char* dx = as.str(1);
+  const char* dy = as.str(2);
   const size_t smem = (size_t)per * 4;
   if (smem > 48 * 1024) cudaFuncSetAttribute(k_mv_rows, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   cudaMemsetAsync(d_err, 0, 8, s);
   k_mv_trunc<<<1, 128, 0, s>>>(c, dy, d_err);
   k_mv_x<<<64, 256, 0, s>>>(c, dx, cols, d_x, d_err);
-  k_mv_rows<<<grid, block, smem, s>>>(c, da, dy, rows, cols, d_x, d_y, d_err);
+  k_mv_rows<<<grid, block, smem, s>>>(c, da, dy, row0, nrows, cols, d_x, d_y, d_err);
   k_mv_sync<<<1, 256, 0, s>>>(c, dy, d_err);
   const cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) fprintf(stderr, "gfs_matvec: launch failed: %s\n", cudaGetErrorString(e));
   return e == cudaSuccess ? 0 : -EIO;
+}
+
+GFS_API int gfs_matvec(gfs_handle* h, void* stream, const char* a_path, const char* x_path, const char* y_path,
+                       uint64_t rows, uint64_t cols, float* d_x, float* d_y, int64_t* d_err, uint32_t grid,
+                       uint32_t block) {
+  return gfs_matvec_rows(h, stream, a_path, x_path, y_path, rows, cols, 0, rows, d_x, d_y, d_err, grid, block);
 }

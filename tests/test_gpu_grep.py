@@ -94,26 +94,61 @@ def test_cache_smaller_than_corpus(g, shmdir):
     assert st["evict"] > 0
 
 
-@pytest.mark.parametrize("chunk", [16, 4096])
-def test_warp_item_scan_vs_oracle(g, shmdir, chunk, monkeypatch):
-    """k_grep_scan_warp (one warp per item, gread_warp; GFS_GREP_WARP=1) is bit-exact too."""
-    monkeypatch.setenv("GFS_GREP_WARP", "1")
-    c = gen.c4_corpus(os.path.join(shmdir, "c4w"), seed=12, nfiles=300, total_bytes=3 << 20, nwords=2000)
+def test_global_file_ids_two_shards(g, shmdir):
+    """A shard grepped with file_ids = its global indices reports global files: the
+    union of two shards' records, their summed totals and their combined digests
+    equal the oracle's over the whole list (hit positions included)."""
+    c = gen.c4_corpus(os.path.join(shmdir, "c4s"), seed=14, nfiles=400, total_bytes=4 << 20, nwords=3000)
     ref = oracle.grep(c["dict"], c["list"], want_hits=True)
-    with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4,
-                 max_files=1024) as fs:
-        out = fs.grep(c["dict"], c["list"], hits=True, chunk=chunk, grid=64)
-    compare(out, ref)
+    from paper_conf_asplos_silbersteinfkw13_b200 import dist as gdist
+    sizes = [os.path.getsize(p) for p in c["paths"]]
+    shards = gdist.lpt_shard(sizes, 2)
+    recs, tot, dsum, dxor, nh, hits = [], 0, 0, 0, 0, []
+    with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4, max_files=1024) as fs:
+        for r, sh in enumerate(shards):
+            lst = gdist.write_shard_list(c["paths"], sh, os.path.join(shmdir, f"shard{r}.txt"))
+            out = fs.grep(c["dict"], lst, hits=True, grid=64, file_ids=np.asarray(sh, np.uint32))
+            assert out["summary"]["err"] == 0
+            recs.append(out["records"])
+            tot = tot + out["totals"].astype(object)
+            dsum, dxor, nh = (dsum + out["digest"][0]) % (1 << 64), dxor ^ out["digest"][1], nh + out["digest"][2]
+            hits.append(out["hits"])
+    allr = np.concatenate(recs)
+    allr = allr[np.lexsort((allr[:, 1], allr[:, 0]))]
+    assert allr.tolist() == ref.records.tolist()
+    assert [int(x) for x in tot] == ref.totals.tolist()
+    assert (dsum, dxor, nh) == tuple(ref.digest)
+    allh = np.concatenate(hits)
+    allh = allh[np.lexsort((allh[:, 2], allh[:, 1], allh[:, 0]))]
+    assert allh.tolist() == ref.hits.tolist()
+
+
+def test_warm_reruns_and_keep_open(g, shmdir):
+    """Back-to-back runs on one work area (the (file, word) table is left empty by
+    each run; keep_open holds files, dictionary and list) stay bit-exact."""
+    c = gen.c4_corpus(os.path.join(shmdir, "c4k"), seed=15, nfiles=300, total_bytes=6 << 20, nwords=2000)
+    ref = oracle.grep(c["dict"], c["list"], want_hits=False)
+    with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4, max_files=1024) as fs:
+        st = fs.grep_state(c["dict"], c["list"], keep_open=True, chunk=4096)
+        for it in range(4):
+            out = fs.grep(c["dict"], c["list"], keep_open=True, chunk=4096, state=st)
+            compare(out, ref, hits=False)
+        s0 = fs.stats()
+        out = fs.grep(c["dict"], c["list"], keep_open=True, chunk=4096, state=st)
+        compare(out, ref, hits=False)
+        assert fs.stats()["rpc_open"] == s0["rpc_open"]  # warm: no open goes to the host
 
 
 def test_max_chunk_and_rejected_chunk(g, shmdir):
     """The largest item (65472 B: item + halos < 64 KiB, 16-bit token offsets) is
-    bit-exact; 65536 is rejected (it overflowed token offsets: wrong counts)."""
+    bit-exact; 65536 is rejected (it overflowed token offsets: wrong counts), and so are
+    chunks that are not multiples of 16."""
     c = gen.c4_corpus(os.path.join(shmdir, "c4m"), seed=13, nfiles=120, total_bytes=4 << 20, nwords=2000)
     ref = oracle.grep(c["dict"], c["list"], want_hits=True)
     with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4,
                  max_files=1024) as fs:
         out = fs.grep(c["dict"], c["list"], hits=True, chunk=65472, grid=64)
         compare(out, ref)
-        with pytest.raises(g.GfsError):
-            fs.grep(c["dict"], c["list"], hits=False, chunk=65536, grid=64)
+        for bad in (65536, 40):
+            with pytest.raises(g.GfsError):
+                fs.grep(c["dict"], c["list"], hits=False, chunk=bad, grid=64)

@@ -131,3 +131,41 @@ def test_checksum_ragged_bytes(shmdir):
     # word 1 = bytes 8..15; take only bytes 10..12 -> value b10<<16 | b11<<24 | b12<<32, weight 3
     expect = (data[10] << 16 | data[11] << 24 | data[12] << 32) * 3
     assert oracle.checksum(path, 10, 3) == expect
+
+
+def _closed_form_checksum(seed, off, ln):
+    """Checksum of bytes [off, off+ln) of a splitmix file from the generator's
+    closed form (SURVEY §8(c) O1 pin 3), byte by byte with Python ints."""
+    if ln == 0:
+        return 0
+    w0, w1 = off // 8, (off + ln - 1) // 8
+    words = gen.splitmix_words(seed, w0, w1 - w0 + 1)
+    s = 0
+    for o in range(off, off + ln):
+        b = (int(words[o // 8 - w0]) >> (8 * (o % 8))) & 0xFF
+        s += (b << (8 * (o % 8))) * (2 * (o // 8) + 1)
+    return s % (1 << 64)
+
+
+def test_checksum_mt_closed_form(shmdir):
+    """The threaded split of the checksum equals the closed form for any cut."""
+    size = 300_000
+    path = gen.splitmix_file(os.path.join(shmdir, "m.bin"), size, seed=5)
+    for off, ln in [(0, size), (3, 77_777), (size - 13, 13), (8, 0), (12345, 99_999)]:
+        expect = _closed_form_checksum(5, off, ln)
+        for t in (1, 2, 3, 7, 16):
+            assert oracle.checksum_mt(path, off, ln, nthreads=t) == expect, (off, ln, t)
+
+
+def test_checksum_calls_closed_form(shmdir):
+    """K4 total = sum over calls of the per-call checksum (repeats included)."""
+    size = 1 << 18
+    path = gen.splitmix_file(os.path.join(shmdir, "k.bin"), size, seed=11)
+    rng = np.random.default_rng(3)
+    chunk = 4096
+    offs = rng.integers(0, size // chunk, size=37) * chunk
+    offs[5] = offs[9]  # a repeated call counts twice
+    expect = sum(_closed_form_checksum(11, int(o), chunk) for o in offs) % (1 << 64)
+    for t in (1, 4):
+        assert oracle.checksum_calls(path, offs, chunk, nthreads=t) == expect
+    assert oracle.checksum_calls(path, [], chunk) == 0
