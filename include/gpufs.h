@@ -159,8 +159,10 @@ int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mode, uint3
  * range of [file_off, file_off + total) in `chunk`-byte calls — gread into
  * d_scratch + b*chunk (use_mmap = 0) or gmmap (use_mmap = 1) — and adds the
  * position-weighted checksum sum_j w_j*(2j+1) of the bytes read (j = global
- * 8-byte word index) into *d_sum. Ranges are split in multiples of chunk.
- * *d_err receives the most negative error seen (0 if none). */
+ * 8-byte word index) into *d_sum. use_mmap = 2: gread only, into
+ * d_scratch + (o - file_off) (a destination of `total` bytes: the cache-hit
+ * gread -> global measurement; *d_sum untouched). Ranges are split in
+ * multiples of chunk. *d_err receives the most negative error seen (0 if none). */
 int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint64_t file_off, uint64_t total,
                     uint64_t chunk, int use_mmap, uint8_t* d_scratch, uint64_t* d_sum, int64_t* d_err,
                     uint32_t grid, uint32_t block);

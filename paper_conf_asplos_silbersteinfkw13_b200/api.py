@@ -122,15 +122,19 @@ class GpuFS:
 
     # sequential sweep (C2 / K1) ---------------------------------------------
     def seqread(self, path, total, chunk, file_off=0, use_mmap=False, grid=296, block=256, stream=None,
-                sync=True, scratch=None, out=None):
+                sync=True, scratch=None, out=None, to_global=False):
+        """Sequential sweep of [file_off, file_off + total) in chunk-byte calls; returns (checksum, err).
+        to_global: gread only, into `scratch` (>= total bytes) at each call's file offset."""
         torch = _torch()
         dev = f"cuda:{self.device}"
+        mode = 2 if to_global else (1 if use_mmap else 0)
         if scratch is None:
-            scratch = torch.empty(max(1, grid * chunk if not use_mmap else 1), dtype=torch.uint8, device=dev)
+            n = total if to_global else (grid * chunk if not use_mmap else 1)
+            scratch = torch.empty(max(1, n), dtype=torch.uint8, device=dev)
         if out is None:
             out = torch.zeros(2, dtype=torch.int64, device=dev)  # [sum, err]
         s, sp = self._stream(stream)
-        gfs_run_seqread(self.h, sp, path, file_off, total, chunk, 1 if use_mmap else 0, scratch.data_ptr(),
+        gfs_run_seqread(self.h, sp, path, file_off, total, chunk, mode, scratch.data_ptr(),
                         out.data_ptr(), out.data_ptr() + 8, grid, block)
         if not sync:
             return out

@@ -1243,7 +1243,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   k_grep_list_emit<<<list_blocks, 256, 0, s>>>(w, p->max_files);
   // gopen is collective with one leader thread: many one-warp blocks keep
   // more opens in flight (host RPCs when cold, L2 round trips when warm)
-  k_grep_open<<<nsm * 32, 32, 0, s>>>(c, w, d_dir, (uint32_t)dir.size(), p->max_files);
+  k_grep_open<<<nsm * 16, 32, 0, s>>>(c, w, d_dir, (uint32_t)dir.size(), p->max_files);
   k_grep_plan<<<1, 1024, 0, s>>>(w);
   k_grep_items<<<nsm * 2, 256, 0, s>>>(w);
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);

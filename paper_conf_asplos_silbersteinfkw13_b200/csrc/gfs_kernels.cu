@@ -182,7 +182,14 @@ __global__ void __launch_bounds__(256, 4) k_seqread(const gfs_ctx* c, const char
   for (uint64_t k = c0; k < c1; ++k) {
     const uint64_t o = file_off + k * chunk;
     const uint64_t want = (k + 1) * chunk <= total ? chunk : total - k * chunk;
-    if (!use_mmap) {
+    if (use_mmap == 2) {  // copy only: gread into the full-size destination at the file offset (cache-hit
+                          // gread -> global: 2 HBM bytes per byte, no consumer pass)
+      const int64_t r = gread(c, fd, o, want, scratch + (o - file_off));
+      if (r < 0) {
+        if (tid == 0) note_err(err, r);
+        break;
+      }
+    } else if (!use_mmap) {
       const int64_t r = gread(c, fd, o, want, buf);
       if (r < 0) {
         if (tid == 0) note_err(err, r);

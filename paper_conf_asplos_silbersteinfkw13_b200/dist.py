@@ -30,6 +30,36 @@ def lpt_shard(sizes, nranks: int) -> list[list[int]]:
     return [sorted(x) for x in out]
 
 
+def row_block(rows: int, nranks: int, rank: int) -> tuple[int, int]:
+    """The contiguous row block [r0, r1) of `rank` in the C3 row split."""
+    return rows * rank // nranks, rows * (rank + 1) // nranks
+
+
+def byte_range(size: int, nranks: int, rank: int, align: int) -> tuple[int, int]:
+    """The byte range [off, off + n) of `rank` in the C2 split of one file (§8(e)):
+    equal `align`-multiple pieces, the last rank takes the rest."""
+    per = (size // nranks) // align * align
+    off = rank * per
+    return off, (size - off if rank == nranks - 1 else per)
+
+
+def gather_rows(pg_world, y_shard, rows: int, device=None):
+    """All-gather of the ranks' y shards (NCCL / gloo all_gather of zero-padded
+    equal-size buffers): the whole y, in row order, on every rank."""
+    import torch
+    import torch.distributed as dist
+    ws = dist.get_world_size(pg_world) if (pg_world is not None and dist.is_initialized()) else 1
+    if ws == 1:
+        return y_shard
+    per = (rows + ws - 1) // ws
+    dev = device if device is not None else y_shard.device
+    yp = torch.zeros(per, dtype=y_shard.dtype, device=dev)
+    yp[:y_shard.numel()] = y_shard
+    parts = [torch.zeros_like(yp) for _ in range(ws)]
+    dist.all_gather(parts, yp, group=pg_world)
+    return torch.cat([parts[r][:row_block(rows, ws, r)[1] - row_block(rows, ws, r)[0]] for r in range(ws)])
+
+
 def write_shard_list(paths, idx, out_path: str) -> str:
     """List file for one shard (absolute paths, one per line)."""
     tmp = out_path + f".tmp{os.getpid()}"
@@ -50,13 +80,20 @@ def globalize_records(records: np.ndarray, shard_idx) -> np.ndarray:
     return r
 
 
-def reduce_grep(pg_world, totals, digest, records, device=None):
+def reduce_grep(pg_world, totals, digest, records, device=None, root=None):
     """The final reduction: all-reduce (sum) of per-word totals, of the hit
-    count and of the order-independent digest sum; all-gather of the XOR
-    terms; gather of the (already global) record arrays to every rank.
-    Works for the NCCL and gloo backends. Returns (totals, digest, records)."""
+    count and of the order-independent digest sum; all-gather of the XOR terms
+    (8 bytes per rank); the (already global) record arrays gathered to `root`
+    (or to every rank when root is None). Works for the NCCL and gloo backends;
+    without a process group (one rank) returns the local values.
+    Returns (totals, digest, records) — records empty on ranks other than root."""
     import torch
     import torch.distributed as dist
+    if pg_world is None or not dist.is_initialized() or dist.get_world_size(pg_world) == 1:
+        recs = np.asarray(records, dtype=np.uint64).reshape(-1, 3)
+        if len(recs):
+            recs = recs[np.lexsort((recs[:, 1], recs[:, 0]))]
+        return (np.asarray(totals, dtype=np.uint64), (int(digest[0]), int(digest[1]), int(digest[2])), recs)
     dev = device if device is not None else torch.device("cpu")
     t = torch.as_tensor(np.asarray(totals, dtype=np.uint64).view(np.int64), device=dev).clone()
     dist.all_reduce(t, op=dist.ReduceOp.SUM, group=pg_world)
@@ -69,11 +106,19 @@ def reduce_grep(pg_world, totals, digest, records, device=None):
     xor = np.uint64(0)
     for v in xs:
         xor ^= np.int64(v.item()).astype(np.uint64)
-    objs = [None] * ws
-    dist.all_gather_object(objs, np.asarray(records, dtype=np.uint64), group=pg_world)
-    recs = np.concatenate([o for o in objs if len(o)]) if any(len(o) for o in objs) else np.zeros((0, 3), np.uint64)
-    if len(recs):
-        recs = recs[np.lexsort((recs[:, 1], recs[:, 0]))]
+    mine = np.asarray(records, dtype=np.uint64)
+    if root is None:
+        objs = [None] * ws
+        dist.all_gather_object(objs, mine, group=pg_world)
+    else:
+        objs = [None] * ws if dist.get_rank() == root else None
+        dist.gather_object(mine, objs, dst=root, group=pg_world)
+    if objs is not None:
+        recs = np.concatenate([o for o in objs if len(o)]) if any(len(o) for o in objs) else np.zeros((0, 3), np.uint64)
+        if len(recs):
+            recs = recs[np.lexsort((recs[:, 1], recs[:, 0]))]
+    else:
+        recs = np.zeros((0, 3), np.uint64)
     tot = t.cpu().numpy().view(np.uint64)
     sv = s.cpu().numpy()
     return tot, (int(np.int64(sv[0]).astype(np.uint64)), int(xor), int(sv[1])), recs

@@ -61,3 +61,48 @@ def test_gloo_world2_reduce_equals_whole(shmdir):
     assert np.load(os.path.join(shmdir, "tot.npy")).tolist() == whole.totals.tolist()
     assert np.load(os.path.join(shmdir, "recs.npy")).tolist() == whole.records.tolist()
     assert int(np.load(os.path.join(shmdir, "nh.npy"))[0]) == whole.digest[2]
+
+
+def _worker_rows(rank, ws, port, m, outdir):
+    import torch
+    import torch.distributed as dist
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=ws)
+    rows, cols = m["rows"], m["cols"]
+    r0, r1 = gdist.row_block(rows, ws, rank)
+    ys = torch.as_tensor(oracle.matvec(m["A"], m["x"], rows, cols, row0=r0, nrows=r1 - r0).astype(np.float32))
+    y = gdist.gather_rows(dist.group.WORLD, ys, rows)
+    # records gathered to rank 0 only
+    recs = np.array([[rank, 1, 2]], dtype=np.uint64)
+    _, _, got = gdist.reduce_grep(dist.group.WORLD, np.zeros(3, np.uint64), (rank, 0, 1), recs, root=0)
+    np.save(os.path.join(outdir, f"y{rank}.npy"), y.numpy())
+    np.save(os.path.join(outdir, f"r{rank}.npy"), got)
+    dist.barrier()
+    dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("ws", [2, 3])
+def test_gloo_row_split_gather_equals_whole(shmdir, ws):
+    """C3 row blocks (one per rank) + all-gather == the whole product; grep records
+    gathered to rank 0 only (the bench's multi-GPU plumbing)."""
+    m = gen.matrix_files(os.path.join(shmdir, "mv"), 37, 96, seed=5)
+    mp.spawn(_worker_rows, args=(ws, _free_port(), m, shmdir), nprocs=ws, join=True)
+    whole = oracle.matvec(m["A"], m["x"], 37, 96).astype(np.float32)
+    for r in range(ws):
+        assert np.array_equal(np.load(os.path.join(shmdir, f"y{r}.npy")), whole)
+    assert np.load(os.path.join(shmdir, "r0.npy")).tolist() == [[r, 1, 2] for r in range(ws)]
+    for r in range(1, ws):
+        assert len(np.load(os.path.join(shmdir, f"r{r}.npy"))) == 0
+
+
+def test_split_helpers_cover_everything():
+    for n in (1, 2, 3, 8):
+        blocks = [gdist.row_block(11200, n, r) for r in range(n)]
+        assert blocks[0][0] == 0 and blocks[-1][1] == 11200
+        assert all(blocks[i][1] == blocks[i + 1][0] for i in range(n - 1))
+        size, P = (8 << 30) + 12345, 2 << 20
+        rngs = [gdist.byte_range(size, n, r, P) for r in range(n)]
+        assert rngs[0][0] == 0 and sum(x[1] for x in rngs) == size
+        assert all(rngs[i][0] + rngs[i][1] == rngs[i + 1][0] for i in range(n - 1))
+        assert all(x[0] % P == 0 for x in rngs)
