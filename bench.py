@@ -799,6 +799,46 @@ def fig4_phase(X, paths, size, h2d):
                         f"mean of {args.fig4_reps}", "points": out}
 
 
+# ---------------------------------------------------------------------- NEXT-2 read-ahead
+def readahead_phase(X, paths, h2d):
+    """NEXT-2: a sequential sweep by few blocks (each block's misses
+    are serialised RPC -> host copy -> pull) with and without read-ahead (the next
+    pages' READ RPCs posted, not waited for, and taken over by the later calls).
+    The first 2 GiB of the two C2 files alternate under a 1 GiB cache: every page
+    a miss. Parity: checksums == the oracle's."""
+    args, torch, g = X.args, X.torch, X.g
+    import oracle
+    total, P = 2 << 30, 2 << 20
+    want = [oracle.checksum_mt(p, 0, total, nthreads=X.nproc) for p in paths] if X.rank == 0 else None
+    want = X.gather(want)[0]
+    pts = []
+    for grid in (8, 32):
+        row = {"grid": grid}
+        for ra in (0, 2):
+            with g.GpuFS(cache_bytes=1 << 30, page_size=P, device=X.local, daemon_threads=args.daemon_threads,
+                         timeout_ms=args.timeout_ms, max_batch=1, readahead=ra) as fs:
+                scratch = torch.empty(grid * P, dtype=torch.uint8, device=X.dev)
+                res = torch.zeros(2, dtype=torch.int64, device=X.dev)
+                ts, ok = [], True
+                for rep in range(1 + args.reps):
+                    t = X.timed(lambda: (res.zero_(), fs.seqread(paths[rep % 2], total, P, grid=grid,
+                                                                 stream=X.stream, sync=False, scratch=scratch,
+                                                                 out=res)), 1)
+                    ok &= (int(res[0].item()) & M64) == want[rep % 2] and int(res[1].item()) == 0
+                    if rep:
+                        ts += t
+                st = fs.stats()
+            m, sd = mstd(ts)
+            row[f"ra{ra}"] = {"GBps": round(gbs(total, m), 3), "GBps_std": round(gbs(total, m) * sd / m, 3),
+                              "frac_h2d": round(gbs(total, m) / h2d, 4), "parity": bool(ok),
+                              "ra_issued": st["ra_issued"], "ra_adopted": st["ra_adopted"],
+                              "ra_reaped": st["ra_reaped"]}
+        row["speedup"] = round(row["ra2"]["GBps"] / row["ra0"]["GBps"], 3)
+        pts.append(row)
+    return {"workload": f"sequential gread sweep of 2 GiB by 8 / 32 blocks, 2 MiB pages, 1 GiB cache, every page "
+                        f"a miss; read-ahead 0 vs 2 pages; mean of {args.reps}", "points": pts}
+
+
 # ---------------------------------------------------------------------- C5
 def c5_phase(X, h2d):
     """C5 (configs[4]): repeated gwrite/gfsync then re-read across kernel launches.
@@ -1035,6 +1075,8 @@ def run_ours(args):
         extra["matvec"] = matvec_phase(X, h2d)
     if not args.no_fig4:
         extra["fig4_page_sweep"] = fig4_phase(X, paths, size, h2d)
+    if not args.no_ra:
+        extra["readahead"] = readahead_phase(X, paths, h2d)
     if not args.no_c5:
         extra["c5"] = c5_phase(X, h2d)
     cpu = cpu_baseline(X, paths[0], size) if (X.rank == 0 and not args.no_cpu) else None
@@ -1114,6 +1156,10 @@ def make_summary(line, c2, extra):
     if f4:
         s["fig4_frac_h2d"] = {p["page_kib"]: p["frac_h2d"] for p in f4["points"]}
         s["fig4_parity"] = all(p["parity"] for p in f4["points"])
+    ra = extra.get("readahead")
+    if ra:
+        s["ra_grid8_GBps"] = [ra["points"][0]["ra0"]["GBps"], ra["points"][0]["ra2"]["GBps"]]
+        s["ra_parity"] = all(p[k]["parity"] for p in ra["points"] for k in ("ra0", "ra2"))
     c5 = extra.get("c5")
     if c5:
         s.update({"c5_write_GBps": c5["write"]["GBps"], "c5_reread_miss_GBps": c5["read_miss"]["GBps"],
@@ -1149,6 +1195,7 @@ def main():
     ap.add_argument("--no-matvec", action="store_true")
     ap.add_argument("--no-c5", action="store_true")
     ap.add_argument("--no-fig4", action="store_true")
+    ap.add_argument("--no-ra", action="store_true", help="skip the read-ahead (NEXT-2) phase")
     ap.add_argument("--no-k1", action="store_true")
     ap.add_argument("--no-split", action="store_true", help="skip the C2 byte-range split (N > 1)")
     ap.add_argument("--no-zc", action="store_true", help="skip the zero-copy (registered file) variants")

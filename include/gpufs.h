@@ -46,7 +46,17 @@ typedef struct gfs_config {
   uint32_t staging_slots;   /* pinned host staging slots of page_size bytes (0 = auto: 128 MiB worth) */
   uint64_t timeout_ms;      /* device-side wait bound (0 = none) -> -ETIMEDOUT */
   void* frame_pool;         /* optional caller-owned device memory >= cache_bytes */
+  uint32_t readahead;       /* NEXT-2: pages a block's sequential gread of a read-only file fetches ahead
+                               (READ RPCs posted, not waited for), 0 = off, at most 8 */
+  uint32_t fault;           /* tests: daemon fault injection, GFS_FAULT_* kind << 24 | period (0 = off) */
 } gfs_config;
+
+/* Daemon fault injection (tests): every `period`-th READ RPC of a
+ * file of at least 2 pages fails with -EIO (GFS_FAULT_EIO) or returns half the
+ * bytes it was asked for (GFS_FAULT_SHORT; the GPU zero-fills the rest, as
+ * for a file that shrank under the cache, R4). */
+#define GFS_FAULT_EIO 1u
+#define GFS_FAULT_SHORT 2u
 
 typedef struct gfs_handle gfs_handle;
 
@@ -184,6 +194,16 @@ int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, con
 int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
                           uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
                           int64_t* d_err, uint32_t grid, uint32_t block);
+
+/* The same benchmark with the split-phase lane-parallel gread (NEXT-2,
+ * gread_lanes_issue / gread_lanes_wait): warp 0 of each block issues the next
+ * `depth` calls (one lane each) into one half of a double buffer of
+ * 2 * depth * chunk bytes of shared memory while the block checksums the other
+ * half. raw: the same schedule with plain TMA copies from d_raw. block: a
+ * multiple of 32, <= 256; depth <= 32; 2 * depth * chunk <= 200 KiB. */
+int gfs_run_randread_async(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
+                           uint32_t chunk, uint32_t calls_per_block, uint32_t depth, const uint64_t* d_off,
+                           uint64_t* d_sum, int64_t* d_err, uint32_t grid, uint32_t block);
 
 /* Write harness: each block gopen(path, flags) — GFS_O_GWRONCE (write-once,
  * diff against zeros) or GFS_O_RDWR (pages fetched, diff against

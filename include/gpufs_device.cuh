@@ -285,7 +285,19 @@ struct Scratch {
   uint32_t lo[GFS_MAX_BATCH], hi[GFS_MAX_BATCH];
   int32_t err;
   uint32_t busy;
+  // read-ahead (NEXT-2), valid for ra_grid / ra_blk: the block's last gread
+  // (fd, end), the highest page fetched ahead, and the fills it posted that
+  // nobody has completed yet (frame, f_pf value), reaped at gclose
+  uint64_t ra_grid;
+  uint32_t ra_blk;
+  int32_t ra_fd;
+  uint64_t ra_next;
+  uint64_t ra_hi;
+  uint32_t ra_n;
+  uint32_t ra_f[16];
+  uint64_t ra_v[16];
 };
+constexpr uint32_t kRA = 16;  // read-ahead fills a block tracks
 
 __device__ __forceinline__ Scratch& scratch() {
   __shared__ Scratch s;
@@ -298,6 +310,7 @@ __device__ __forceinline__ Scratch& scratch() {
 // its scratch lives. key() identifies the group within a launch (scratch is
 // shared memory, never cleared, so cached state is keyed by grid and group).
 struct BlockGroup {
+  static constexpr bool kBlock = true;
   static __device__ __forceinline__ int tid() { return block_tid(); }
   static __device__ __forceinline__ int nthr() { return block_nthr(); }
   static __device__ __forceinline__ void sync() { __syncthreads(); }
@@ -313,6 +326,7 @@ __device__ __forceinline__ Scratch& warp_scratch(int w) {
   return s[w];
 }
 struct WarpGroup {  // every lane of the calling warp takes part (full warps only)
+  static constexpr bool kBlock = false;
   static __device__ __forceinline__ int tid() { return block_tid() & 31; }
   static __device__ __forceinline__ int nthr() { return 32; }
   static __device__ __forceinline__ void sync() { __syncwarp(); }
@@ -364,9 +378,10 @@ __device__ __forceinline__ uint8_t* stage_ptr(const gfs_ctx* c, int idx) {
 // slot in pinned host memory, publish seq with st.release.sys (the GPU->CPU
 // fence), then poll the completion word the host stores in pinned
 // memory (ld.acquire.sys: P:L693-696's cache bypass). Any thread may call.
-__device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64_t file_off, int stage,
-                            uint32_t len, uint32_t flags, uint64_t arg, const char* path, uint32_t path_len,
-                            gfs_rpc_resp* resp_out) {
+// rpc_post + rpc_complete are the two halves (read-ahead posts and lets any
+// thread complete later); rpc_call is both. Returns the ticket, or -ETIMEDOUT.
+__device__ int64_t rpc_post(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64_t file_off, int stage, uint32_t len,
+                            uint32_t flags, uint64_t arg, const char* path, uint32_t path_len) {
   const unsigned long long t = atom_add64(c->ring_tail, 1ull);
   const uint32_t R = c->ring_slots;
   const uint32_t slot = (uint32_t)(t % R);
@@ -407,9 +422,17 @@ __device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64
   }
   st_rel_sys64((uint64_t*)&q->seq, (uint64_t)(t + 1));
   ctr(c, GFS_C_RPC);
+  return (int64_t)t;
+}
+
+// Wait for ticket t's completion, read its result (and the reply record), and
+// release the ring slot to the ticket's successor.
+__device__ int32_t rpc_complete(const gfs_ctx* c, uint64_t t, gfs_rpc_resp* resp_out) {
+  const uint32_t slot = (uint32_t)(t % c->ring_slots);
   const uint32_t want = (uint32_t)(t + 1);
+  const uint64_t t0 = now_ns();
   uint64_t v;
-  ns = 256;
+  uint32_t ns = 256;
   while (((v = ld_acq_sys64(&c->cpl[slot])) >> 32) != want) {
     backoff(ns);
     if (timed_out(c, t0)) {
@@ -432,6 +455,14 @@ __device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64
   }
   st_rel64(&c->ack[slot], (uint64_t)(t + 1));
   return res;
+}
+
+__device__ int32_t rpc_call(const gfs_ctx* c, uint32_t op, uint32_t hfid, uint64_t file_off, int stage,
+                            uint32_t len, uint32_t flags, uint64_t arg, const char* path, uint32_t path_len,
+                            gfs_rpc_resp* resp_out) {
+  const int64_t t = rpc_post(c, op, hfid, file_off, stage, len, flags, arg, path, path_len);
+  if (t < 0) return (int32_t)t;
+  return rpc_complete(c, (uint64_t)t, resp_out);
 }
 
 // ------------------------------------------------------------------ radix nodes
@@ -815,7 +846,8 @@ __device__ __forceinline__ uint32_t frame_tier(const gfs_ctx* c, uint32_t f, uin
 // writing back a dirty victim first. Runs in the calling thread.
 // Returns the frame in state FILLING|1 with its tag set (and its new
 // generation in *gen), or -ENOMEM.
-__device__ __noinline__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx, uint32_t* gen) {
+__device__ __noinline__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t fdx, uint32_t* gen,
+                                        bool nowait = false) {
   const uint32_t N = c->nframes;
   if (ld_rlx(c->fresh_next) < N) {
     const uint32_t f = atomicAdd(c->fresh_next, 1u);
@@ -831,18 +863,36 @@ __device__ __noinline__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t
     const uint32_t w = atomicAdd(c->hand, 32u);
     int best = -1;
     uint64_t best_key = ~0ull;
-    uint64_t best_st = 0;
+    uint64_t best_st = 0, best_pv = 0;
 #pragma unroll 4
     for (uint32_t j = 0; j < 32; ++j) {
       const uint32_t f = (uint32_t)(((uint64_t)w + j) % N);
       const uint64_t st = ld_rlx64(&c->f_state[f]);
-      if ((uint32_t)st & ~GFS_ST_ERROR) continue;  // referenced, filling or being evicted
-      const uint64_t key = ((uint64_t)frame_tier(c, f, (uint32_t)st) << 32) | ld_rlx(&c->f_stamp[f]);
+      uint64_t pv = 0;
+      if ((uint32_t)st & ~GFS_ST_ERROR) {  // referenced, filling or being evicted ...
+        // ... except a read-ahead fill nobody has asked for yet (NEXT-2): the
+        // last resort (tier 4), so read-ahead never starves a reader of frames
+        if (!c->readahead || (uint32_t)st != GFS_ST_FILLING) continue;
+        pv = ld_rlx64(&c->f_pf[f]);
+        if (pv == 0 || pv == GFS_PF_POSTING) continue;
+      }
+      const uint64_t key =
+          ((uint64_t)(pv ? 4u : frame_tier(c, f, (uint32_t)st)) << 32) | ld_rlx(&c->f_stamp[f]);
       if (key < best_key) {
         best_key = key;
         best = (int)f;
         best_st = st;
+        best_pv = pv;
       }
+    }
+    if (best >= 0 && best_pv) {  // take the unneeded read-ahead fill over and drop its page
+      if (a64_cas(&c->f_pf[best], best_pv, 0) != best_pv) continue;  // someone adopted it meanwhile
+      (void)rpc_complete(c, (best_pv >> 32) - 1, nullptr);  // the slot and ring entry are released first
+      stage_free(c, (int)(uint32_t)best_pv - 1);
+      a64_add_rel(&c->f_state[best], (uint64_t)GFS_ST_EVICTING - (uint64_t)GFS_ST_FILLING);  // keeps transient refs
+      ctr(c, GFS_C_EVICT);
+      *gen = frame_init(c, (uint32_t)best, tag, fdx);
+      return best;
     }
     if (best >= 0 &&
         a64_cas(&c->f_state[best], best_st, (best_st & 0xFFFFFFFF00000000ull) | GFS_ST_EVICTING) == best_st) {
@@ -859,6 +909,7 @@ __device__ __noinline__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t
       *gen = frame_init(c, f, tag, fdx);
       return (int)f;
     }
+    if (nowait && round >= 8) return -EAGAIN;  // read-ahead: a few windows, never wait for a victim
     if (round > 0 && round % windows == 0) {
       backoff(ns);
       if (now_ns() - t0 > 2000000000ull) {  // 2 s of full scans: the deadlock guard
@@ -1085,10 +1136,31 @@ __device__ __noinline__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint
       // same generation as the slot <=> the frame still holds this page (the
       // tag check is kept as a belt-and-braces test on the slow path)
       if ((old >> 32) == (s >> 32) && ld_acq64(&c->f_tag[f]) == want) {
+        uint64_t pv = 0;
         if (!((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
           ctr(c, GFS_C_HIT);
           out.frame = (int)f;
           done = true;
+        } else if (!lk && ((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING)) == GFS_ST_FILLING &&
+                   (pv = ld_acq64(&c->f_pf[f])) != 0 && pv != GFS_PF_POSTING && a64_cas(&c->f_pf[f], pv, 0) == pv) {
+          // a read-ahead fill nobody waits for yet (NEXT-2): this lane completes
+          // it — the host has (or will have) the page in the posted staging
+          // slot — and keeps the reference it just took as its own
+          const int stg = (int)(uint32_t)pv - 1;
+          const int32_t r = rpc_complete(c, (pv >> 32) - 1, nullptr);
+          if (r < 0) {  // the fetch failed: the frame becomes stale, retried below like any stale slot
+            stage_free(c, stg);
+            a64_or_rel(&c->f_state[f], GFS_ST_ERROR);
+            a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));
+            a64_add_rel(&c->f_state[f], kRefDec);
+          } else {
+            ctr(c, GFS_C_RA_ADOPTED);
+            out.frame = (int)f;
+            out.fill = 1;
+            out.stage = stg;
+            out.nbytes = (uint32_t)r;
+            done = true;
+          }
         } else if ((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING)) {  // someone else is on it
           a64_add_rel(&c->f_state[f], kRefDec);
           ctr(c, GFS_C_BUSY);
@@ -1296,6 +1368,195 @@ __device__ int acquire_batch(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, 
       G::sync();
     }
   }
+}
+
+// ------------------------------------------------------------------ read-ahead (NEXT-2)
+// "read-ahead, data transfer scheduling, and asynchronous writes".
+// A block whose gread continues where its previous gread on the same read-only
+// file ended fetches the next c->readahead pages: each is installed (FILLING,
+// no reference held) and its READ RPC posted, but nobody waits. The fill
+// belongs to whoever completes it: the first lookup that needs the page takes
+// it over in lookup_try (waits for the RPC, pulls the page, publishes it), and
+// the issuing block reaps the ones nobody needed at its gclose. No lane ever
+// waits for the issuing block itself, so read-ahead adds no wait-for edge
+// between blocks (the host completes every RPC on its own).
+
+// Post the read-ahead fetch of `page` (< the file's page count). Returns the
+// frame, or -1 when the page is cached / in flight or no slot / frame is free.
+__device__ __noinline__ int ra_issue(const gfs_ctx* c, const FileSnap& fs, uint64_t page, uint64_t* pv_out) {
+  const int f0 = lookup_fast(c, fs, page, nullptr);
+  if (f0 >= 0) {  // cached
+    r64_add_rlx(&c->f_state[f0], kRefDec);
+    return -1;
+  }
+  if (peek_busy(c, fs, page)) return -1;
+  const uint64_t base = page << c->page_shift;
+  const uint64_t rem = fs.size - base;
+  const uint32_t nb = (uint32_t)(rem < c->page_size ? rem : c->page_size);
+  const int st = stage_alloc(c, false);
+  if (st < 0) return -1;
+  uint64_t* slot = walk(c, fs.root, fs.height, page, true, nullptr);
+  if (!slot) {
+    stage_free(c, st);
+    return -1;
+  }
+  const uint64_t s = ld_acq64(slot);
+  if ((uint32_t)s) {  // only a stale slot (frame reassigned, or failed and not refilling) is replaced
+    const uint64_t fst = ld_acq64(&c->f_state[(uint32_t)s - 1u]);
+    const bool stale = (fst >> 32) != (s >> 32) ||
+                       (((uint32_t)fst & GFS_ST_ERROR) && !((uint32_t)fst & GFS_ST_FILLING));
+    if (!stale) {
+      stage_free(c, st);
+      return -1;
+    }
+  }
+  uint32_t gen = 0;
+  const int g = alloc_frame(c, ((uint64_t)fs.uid << 32) | (uint32_t)page, fs.fdx, &gen, true);
+  if (g < 0) {
+    stage_free(c, st);
+    return -1;
+  }
+  st_rel64(&c->f_pf[g], GFS_PF_POSTING);  // lookups that find it now wait (busy) instead of adopting
+  if (a64_cas(slot, s, slot_val((uint32_t)g, gen)) != s) {
+    st_rlx64(&c->f_pf[g], 0);
+    frame_abandon(c, (uint32_t)g);
+    stage_free(c, st);
+    return -1;
+  }
+  a64_add_rel(&c->f_state[g], kRefDec);  // FILLING, unreferenced: the fill is anyone's to complete
+  const int64_t t = rpc_post(c, GFS_OP_READ, fs.hfid, base, st, nb, 0, 0, nullptr, 0);
+  if (t < 0) {  // not posted: the frame fails (a later lookup installs over it)
+    st_rlx64(&c->f_pf[g], 0);
+    stage_free(c, st);
+    a64_or_rel(&c->f_state[g], GFS_ST_ERROR);
+    a64_and_rel(&c->f_state[g], fl64(GFS_ST_FILLING));
+    return -1;
+  }
+  const uint64_t pv = ((uint64_t)(t + 1) << 32) | (uint32_t)(st + 1);
+  st_rel64(&c->f_pf[g], pv);
+  *pv_out = pv;
+  ctr(c, GFS_C_RA_ISSUED);
+  ctr(c, GFS_C_MISS);
+  ctr(c, GFS_C_RPC_READ);
+  ctr(c, GFS_C_BYTES_H2D, nb);
+  return g;
+}
+
+// After a block gread of [off, off + n) on read-only fd (warp 0 only): if it
+// continued the block's previous gread on fd, post the fetches of the pages
+// after it that are not fetched yet (up to c->readahead ahead), and forget
+// the posted fills that other lookups completed meanwhile.
+template <class G>
+__device__ __noinline__ void ra_after(const gfs_ctx* c, Scratch& sc, const FileSnap& fs, int fd, uint64_t off,
+                                      uint64_t n) {
+  const int lane = block_tid() & 31;
+  if (lane == 0 && (sc.ra_grid != grid_id() || sc.ra_blk != G::key())) {
+    sc.ra_grid = grid_id();
+    sc.ra_blk = G::key();
+    sc.ra_fd = -1;
+    sc.ra_n = 0;
+    sc.ra_hi = 0;
+    sc.ra_next = 0;
+  }
+  __syncwarp();
+  const bool seq = sc.ra_fd == fd && sc.ra_next == off;
+  const uint64_t p1 = (off + n - 1) >> c->page_shift;
+  const uint64_t np = (fs.size + c->page_size - 1) >> c->page_shift;
+  // keep the posted fills still pending (f_pf unchanged)
+  const uint32_t n0 = sc.ra_n;
+  bool keep = false;
+  uint32_t kf = 0;
+  uint64_t kv = 0;
+  if ((uint32_t)lane < n0) {
+    kf = sc.ra_f[lane];
+    kv = sc.ra_v[lane];
+    keep = ld_rlx64(&c->f_pf[kf]) == kv;
+  }
+  const uint32_t kb = __ballot_sync(0xFFFFFFFFu, keep);
+  __syncwarp();
+  if (keep) {
+    const uint32_t k = __popc(kb & ((1u << lane) - 1u));
+    sc.ra_f[k] = kf;
+    sc.ra_v[k] = kv;
+  }
+  uint32_t nk = __popc(kb);
+  uint64_t hi = seq ? sc.ra_hi : p1;
+  if (seq) {
+    const uint64_t lo = (sc.ra_hi > p1 ? sc.ra_hi : p1) + 1;
+    uint64_t top = p1 + c->readahead;
+    if (top > np - 1) top = np - 1;
+    const uint64_t pg = lo + (uint64_t)lane;
+    int g = -1;
+    uint64_t pv = 0;
+    if (lo <= top && pg <= top && nk + (uint32_t)lane < kRA) g = ra_issue(c, fs, pg, &pv);
+    const uint32_t ib = __ballot_sync(0xFFFFFFFFu, g >= 0);
+    __syncwarp();
+    if (g >= 0) {
+      const uint32_t k = nk + __popc(ib & ((1u << lane) - 1u));
+      sc.ra_f[k] = (uint32_t)g;
+      sc.ra_v[k] = pv;
+    }
+    nk += __popc(ib);
+    if (lo <= top && top > hi) hi = top;
+  }
+  __syncwarp();
+  if (lane == 0) {
+    sc.ra_n = nk;
+    sc.ra_fd = fd;
+    sc.ra_next = off + n;
+    sc.ra_hi = hi;
+  }
+  __syncwarp();
+}
+
+// At gclose (block-collective): complete every fill this block posted that is
+// still pending — pull the page into its frame and publish it — so no frame
+// stays FILLING and no staging or ring slot stays held after the block is gone.
+template <class G>
+__device__ __noinline__ void ra_reap(const gfs_ctx* c, Scratch& sc) {
+  const int tid = G::tid(), nthr = G::nthr();
+  if (!(sc.ra_grid == grid_id() && sc.ra_blk == G::key()) || sc.ra_n == 0) return;  // uniform: shared values
+  const uint32_t n = sc.ra_n;
+  if (tid < (int)n) {
+    const uint32_t f = sc.ra_f[tid];
+    const uint64_t v = sc.ra_v[tid];
+    sc.frame[tid] = -1;
+    if (a64_cas(&c->f_pf[f], v, 0) == v) {
+      const int st = (int)(uint32_t)v - 1;
+      const int32_t r = rpc_complete(c, (v >> 32) - 1, nullptr);
+      if (r < 0) {
+        stage_free(c, st);
+        a64_or_rel(&c->f_state[f], GFS_ST_ERROR);
+        a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));
+      } else {
+        sc.frame[tid] = (int)f;
+        sc.stage[tid] = st;
+        sc.nbytes[tid] = (uint32_t)r;
+      }
+    }
+  }
+  G::sync();
+  for (uint32_t i = 0; i < n; ++i)
+    if (sc.frame[i] >= 0)
+      block_copy_from_frame<true>(frame_ptr(c, (uint32_t)sc.frame[i]), stage_ptr(c, sc.stage[i]), sc.nbytes[i], tid,
+                                  nthr);
+  if (c->flags & GFS_F_EXPORTED) __threadfence_system();
+  else __threadfence();
+  G::sync();
+  if (tid < (int)n && sc.frame[tid] >= 0) {
+    const uint32_t f = (uint32_t)sc.frame[tid];
+    stage_free(c, sc.stage[tid]);
+    st_rlx(&c->f_valid[f], sc.nbytes[tid]);
+    st_rlx(&c->f_hv[f], sc.nbytes[tid]);
+    st_rlx(&c->f_stamp[f], stamp_now());
+    a64_and_rel(&c->f_state[f], fl64(GFS_ST_FILLING));  // publish: FILLING -> plain unreferenced page
+    ctr(c, GFS_C_RA_REAPED);
+  }
+  if (tid == 0) {
+    sc.ra_n = 0;
+    sc.ra_fd = -1;
+  }
+  G::sync();
 }
 
 // O_RDWR write-back with the diff done on the GPU: for frame f
@@ -1848,6 +2109,9 @@ template <class G>
 __device__ inline int gclose_t(const gfs_ctx* c, int fd) {
   Scratch& sc = G::sc();
   G::sync();
+  if constexpr (G::kBlock) {
+    if (c->readahead) detail::ra_reap<G>(c, sc);  // the block's read-ahead fills nobody completed
+  }
   if (G::tid() == 0) {
     if (sc.cached_fd == fd) sc.cached_fd = -1;
     sc.ret = detail::close_leader(c, fd);
@@ -2008,6 +2272,7 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
   G::sync();
   const int64_t n = sc.ret;
   if (n <= 0) return n;
+  int64_t res = n;
   if (sc.quick) {
     const uint32_t ph = sc.mbar_phase;
     copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + (off & (P - 1)), (uint32_t)n, tid);
@@ -2017,9 +2282,15 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
       sc.mbar_phase = ph ^ 1u;
       frame_release(c, (uint32_t)sc.frame[0]);
     }
-    return n;
+  } else {
+    res = gread_batches<G>(c, n, off, dst);
   }
-  return gread_batches<G>(c, n, off, dst);
+  if constexpr (G::kBlock) {  // NEXT-2: read-ahead of a sequential reader of a read-only file (warp 0)
+    if (c->readahead && res > 0 && tid < 32 && !(sc.fs.oflags & GFS_O_WRITABLE) && !c->npeers &&
+        ld_rlx64(&c->files[sc.fs.fdx].zc) == 0)
+      ra_after<G>(c, sc, sc.fs, fd, off, (uint64_t)res);
+  }
+  return res;
 }
 
 // Threadblock-collective calls (the prototype's granularity).

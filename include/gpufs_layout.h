@@ -57,6 +57,7 @@ extern "C" {
 #define GFS_TAG_NONE 0xFFFFFFFFFFFFFFFFull /* tag = (uid << 32) | page index */
 #define GFS_DIRTY_NONE 0xFFFFFFFFu
 #define GFS_PRISTINE_PENDING 0xFFFFFFFFu
+#define GFS_PF_POSTING 0xFFFFFFFFFFFFFFFFull /* f_pf: read-ahead frame installed, its RPC not posted yet */
 
 /* ---- file table entry states (high byte of `sr`; low 24 bits = refcount) */
 #define GFS_FS_FREE 0u
@@ -165,6 +166,9 @@ enum {
   GFS_C_BYTES_PEER,     /* bytes copied from peer caches */
   GFS_C_PEER_MISS,      /* misses for which no peer held a usable copy */
   GFS_C_ZC_FILL,        /* misses filled straight from a registered file mapping (no RPC) */
+  GFS_C_RA_ISSUED,      /* read-ahead fetches posted (NEXT-2) */
+  GFS_C_RA_ADOPTED,     /* read-ahead fills completed by a lookup that needed the page */
+  GFS_C_RA_REAPED,      /* read-ahead fills completed by their issuer's gclose (page not read meanwhile) */
   GFS_C_NCOUNTERS
 };
 
@@ -238,7 +242,10 @@ typedef struct gfs_ctx {
   /* peer caches (device array of npeers views) */
   const gfs_peer* peers;
   uint32_t npeers;
-  uint32_t pad_peers;
+  uint32_t readahead;  /* pages fetched ahead of a block's sequential gread of a read-only file (0 = off) */
+  /* read-ahead (NEXT-2): per frame, a fill in flight that no reader waits for yet:
+   * 0 none, GFS_PF_POSTING being posted, else ((ticket + 1) << 32) | (staging slot + 1) */
+  uint64_t* f_pf;
 } gfs_ctx;
 
 #ifdef __cplusplus

@@ -18,7 +18,8 @@ LIB_PATH = os.path.join(_PKG, "libgpufs.so")
 COUNTERS = ["hit", "miss", "zero_fill", "lockfree", "locked", "retry", "evict", "writeback", "rpc",
             "rpc_open", "rpc_read", "rpc_write", "bytes_h2d", "bytes_d2h", "open_fast", "reopen_valid",
             "invalidate", "enomem", "timeout", "gread_calls", "gread_bytes", "gwrite_calls", "nodes",
-            "ring_wait", "busy", "stage_wait", "peer_fill", "bytes_peer", "peer_miss", "zc_fill"]
+            "ring_wait", "busy", "stage_wait", "peer_fill", "bytes_peer", "peer_miss", "zc_fill",
+            "ra_issued", "ra_adopted", "ra_reaped"]
 HOST_COUNTERS = ["rpc", "read", "write", "open", "close", "trunc", "bytes_h2d", "bytes_d2h", "pread_ns",
                  "errors", "merges", "busy_ns", "open_ns", "open_sys_ns", "open_prefetch_ns", "open_table_ns",
                  "mapped_reads", "open_vt_ns"]
@@ -28,6 +29,8 @@ O_GWRONCE = 1
 O_RDWR = 2
 PROT_WRITE = 2
 F_LOCKED_TRAVERSAL = 1
+FAULT_EIO = 1    # gfs_config.fault kinds (tests): a READ fails with -EIO
+FAULT_SHORT = 2  # ... or comes back with half its bytes
 F_NO_DMA_COMPLETION = 2
 DAEMON_SPAWN = 0
 DAEMON_RUN = 1
@@ -42,7 +45,7 @@ class gfs_config(ctypes.Structure):
                 ("ring_slots", ctypes.c_uint32), ("daemon_threads", ctypes.c_uint32),
                 ("max_files", ctypes.c_uint32), ("max_nodes", ctypes.c_uint32), ("max_batch", ctypes.c_uint32),
                 ("flags", ctypes.c_uint32), ("staging_slots", ctypes.c_uint32), ("timeout_ms", ctypes.c_uint64),
-                ("frame_pool", ctypes.c_void_p)]
+                ("frame_pool", ctypes.c_void_p), ("readahead", ctypes.c_uint32), ("fault", ctypes.c_uint32)]
 
 
 class gfs_grep_params(ctypes.Structure):
@@ -92,6 +95,7 @@ def lib():
             "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_randread_warp": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
+            "gfs_run_randread_async": ([P, P, CS, I, P, U32, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32, I], I),
             "gfs_run_mmap_write": ([P, P, CS, U32, P, P, P, P, P, U32, U32, I], I),
             "gfs_run_fileop": ([P, P, CS, I, I, U64, P], I),
@@ -201,6 +205,12 @@ def gfs_run_seqread(h, stream, path, file_off, total, chunk, use_mmap, d_scratch
 def gfs_run_randread(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):
     return _ck(lib().gfs_run_randread(h, stream, _b(path) if path else None, raw, d_raw, chunk, calls_per_block,
                                       d_off, d_sum, d_err, grid, block), "gfs_run_randread")
+
+
+def gfs_run_randread_async(h, stream, path, raw, d_raw, chunk, calls_per_block, depth, d_off, d_sum, d_err, grid,
+                           block):
+    return _ck(lib().gfs_run_randread_async(h, stream, _b(path) if path else None, raw, d_raw, chunk, calls_per_block,
+                                            depth, d_off, d_sum, d_err, grid, block), "gfs_run_randread_async")
 
 
 def gfs_run_randread_warp(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):

@@ -24,7 +24,8 @@ class GpuFS:
     """One GPU buffer cache + its host daemon (gfs_init + gfs_daemon)."""
 
     def __init__(self, cache_bytes=1 << 30, page_size=64 << 10, device=0, daemon_threads=8, ring_slots=4096,
-                 max_files=4096, max_nodes=0, max_batch=32, flags=0, timeout_ms=60000, staging_slots=0):
+                 max_files=4096, max_nodes=0, max_batch=32, flags=0, timeout_ms=60000, staging_slots=0,
+                 readahead=0, fault=0):
         torch = _torch()
         torch.cuda.set_device(device)
         self.device = device
@@ -32,7 +33,7 @@ class GpuFS:
         cfg = gfs_config_default(device=device, cache_bytes=cache_bytes, page_size=page_size,
                                  daemon_threads=daemon_threads, ring_slots=ring_slots, max_files=max_files,
                                  max_nodes=max_nodes, max_batch=max_batch, flags=flags, timeout_ms=timeout_ms,
-                                 staging_slots=staging_slots)
+                                 staging_slots=staging_slots, readahead=readahead, fault=fault)
         self.h = gfs_init(cfg)
         gfs_daemon(self.h, DAEMON_SPAWN)
 
@@ -161,7 +162,10 @@ class GpuFS:
         return int(out[0].item())
 
     # cache-hit reads into shared memory (K4) ---------------------------------
-    def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None, warp=False):
+    def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None, warp=False,
+                 depth=0):
+        """K4 reads into shared memory; warp: the warp-collective calls; depth > 0: the split-phase
+        lane-parallel calls, `depth` of them in flight per block (gfs_run_randread_async)."""
         torch = _torch()
         dev = f"cuda:{self.device}"
         if isinstance(offs, torch.Tensor):
@@ -173,7 +177,16 @@ class GpuFS:
         if out is None:
             out = torch.zeros(2, dtype=torch.int64, device=dev)
         s, sp = self._stream(stream)
-        from . import gfs_run_randread_warp
+        from . import gfs_run_randread_async, gfs_run_randread_warp
+        if depth:
+            gfs_run_randread_async(self.h, sp, path, 1 if raw is not None else 0,
+                                   raw.data_ptr() if raw is not None else None, chunk, calls, depth,
+                                   d_off.data_ptr(), out.data_ptr(), out.data_ptr() + 8, grid, block)
+            if not sync:
+                return out
+            s.synchronize()
+            v = out.cpu().numpy()
+            return int(v[0].astype(np.uint64)), int(v[1])
         fn = gfs_run_randread_warp if warp else gfs_run_randread
         fn(self.h, sp, path, 1 if raw is not None else 0,
                          raw.data_ptr() if raw is not None else None, chunk, calls, d_off.data_ptr(),

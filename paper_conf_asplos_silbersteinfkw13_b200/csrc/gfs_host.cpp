@@ -255,6 +255,7 @@ struct gfs_handle {
   SpinMutex zc_mu;
   std::vector<ZcFile> zc;
   std::vector<void*> ipc_open;   // CUDA IPC mappings to close at shutdown
+  std::atomic<uint64_t> fault_ctr{0};  // READs seen by the fault injector (gfs_config.fault)
   // Launcher argument staging (path strings for the kernels): a ring of slots
   // in pinned host + device memory of this handle's device. A slot is reused
   // only after the event recorded behind the LAST kernel that read it.
@@ -594,6 +595,14 @@ const uint8_t* hfid_map(gfs_handle* h, Worker& w, uint32_t id, uint64_t* map_len
 int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
   if (q.len > h->h.page_size || q.stage >= h->h.staging_slots) return -EINVAL;
   uint8_t* buf = staging_slot(h, q.stage);
+  uint32_t qlen = q.len;
+  if (h->cfg.fault) {  // tests: every period-th READ past a file's first page fails or comes back short
+    const uint32_t kind = h->cfg.fault >> 24, period = h->cfg.fault & 0xFFFFFFu;
+    if (period && q.file_off >= h->h.page_size && h->fault_ctr.fetch_add(1) % period == period - 1) {
+      if (kind == GFS_FAULT_EIO) return -EIO;
+      if (kind == GFS_FAULT_SHORT) qlen = q.len / 2;  // as if the file ended there: the rest reads as zeros
+    }
+  }
   auto t0 = std::chrono::steady_clock::now();
   uint64_t map_len = 0;
   const uint8_t* map = hfid_map(h, w, q.hfid, &map_len);
@@ -605,13 +614,13 @@ int32_t do_read(gfs_handle* h, Worker& w, const gfs_rpc_req& q) {
     }
   }
   int64_t n = -1;
-  if (map && q.file_off + q.len <= map_len && map_copy(buf, map, q.file_off, q.len)) {
-    n = q.len;
+  if (map && q.file_off + qlen <= map_len && map_copy(buf, map, q.file_off, qlen)) {
+    n = qlen;
     w.add(HS_MAPPED, 1);
   } else {
     const int fd = w_fd(h, w, q.hfid);
     if (fd < 0) return fd;
-    n = pread_full(fd, buf, q.len, q.file_off);
+    n = pread_full(fd, buf, qlen, q.file_off);
   }
   w.add(HS_PREAD_NS, (uint64_t)std::chrono::duration_cast<std::chrono::nanoseconds>(
                             std::chrono::steady_clock::now() - t0).count());
@@ -890,7 +899,7 @@ void free_all(gfs_handle* h) {
   h->ipc_open.clear();
   if (h->own_pool) F(h->h.pool);
   F(h->h.f_state); F(h->h.f_tag); F(h->h.f_file); F(h->h.f_valid); F(h->h.f_lo); F(h->h.f_hi);
-  F(h->h.f_written); F(h->h.f_stamp); F(h->h.f_hv); F(h->h.f_pristine); F((void*)h->h.peers); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
+  F(h->h.f_written); F(h->h.f_stamp); F(h->h.f_hv); F(h->h.f_pristine); F(h->h.f_pf); F((void*)h->h.peers); F(h->h.fresh_next); F(h->h.hand); F(h->h.nodes); F(h->h.node_next);
   F(h->h.node_free); F(h->h.node_free_top); F(h->h.node_lock); F(h->h.files); F(h->h.paths); F(h->h.uid_next);
   F(h->h.ack); F(h->h.ring_tail); F(h->h.ctr); F(h->h.staging_bits); F(h->d);
   if (h->ring_h) cudaFreeHost(h->ring_h);
@@ -993,6 +1002,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMalloc((void**)&c.f_stamp, nframes * 4));
   CK(cudaMalloc((void**)&c.f_hv, nframes * 4));
   CK(cudaMalloc((void**)&c.f_pristine, nframes * 4));
+  CK(cudaMalloc((void**)&c.f_pf, nframes * 8));
   CK(cudaMalloc((void**)&c.fresh_next, 4));
   CK(cudaMalloc((void**)&c.hand, 4));
   c.max_nodes = max_nodes;
@@ -1027,6 +1037,7 @@ GFS_API int gfs_init(const gfs_config* cfg, gfs_handle** out) {
   CK(cudaMalloc((void**)&c.ring_tail, 8));
   CK(cudaMalloc((void**)&c.ctr, ctr_bytes));
   c.flags = cfg->flags;
+  c.readahead = cfg->readahead <= 8 ? cfg->readahead : 8;
   c.max_batch = cfg->max_batch >= 1 && cfg->max_batch <= GFS_MAX_BATCH ? cfg->max_batch : GFS_MAX_BATCH;
   c.timeout_ns = cfg->timeout_ms * 1000000ull;
   CK(cudaMemsetAsync(c.nodes, 0, (size_t)max_nodes * GFS_FANOUT * 8, h->priv));

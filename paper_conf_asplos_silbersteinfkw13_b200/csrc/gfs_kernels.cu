@@ -36,6 +36,7 @@ __global__ void k_init_metadata(gfs_ctx c) {
     c.f_stamp[i] = 0;
     c.f_hv[i] = 0;
     c.f_pristine[i] = 0;
+    c.f_pf[i] = 0;
   }
   if (blockIdx.x == 0 && threadIdx.x == 0) {
     *c.fresh_next = 0;
@@ -320,6 +321,74 @@ __global__ void __launch_bounds__(256) k_randread_warp(const gfs_ctx* c, const c
   if (!raw) gclose_warp(c, fd);
 }
 
+// K4 with the split-phase lane-parallel gread (NEXT-2): warp 0 issues the
+// block's next `depth` calls (one lane each: lookups and TMA copies in flight)
+// into one half of a double buffer while the whole block checksums the other
+// half, so a call's page-table walk and copy overlap the previous calls'
+// consumption. raw: the same schedule with plain TMA copies of d_raw.
+__global__ void __launch_bounds__(256) k_randread_async(const gfs_ctx* c, const char* path, int raw,
+                                                        const uint8_t* rawp, uint32_t chunk, uint32_t calls,
+                                                        uint32_t depth, const uint64_t* offs, uint64_t* sum,
+                                                        int64_t* err) {
+  extern __shared__ __align__(16) uint8_t smem[];
+  __shared__ uint64_t raw_mbar;
+  const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31, wid = tid >> 5;
+  int fd = 0;
+  if (!raw) {
+    fd = gopen(c, path, GFS_O_RDONLY);  // block-collective; the warp calls below use it
+    if (fd < 0) {
+      if (tid == 0) note_err(err, fd);
+      return;
+    }
+  } else if (tid == 0) {
+    detail::mbar_init(&raw_mbar);
+  }
+  __syncthreads();
+  const uint64_t* my = offs + (size_t)blockIdx.x * calls;
+  GreadLaneTicket tk{0, -1, -1, 0, 0};
+  uint32_t raw_ph = 0;
+  // issue calls [base, base + depth) into half h (warp 0)
+  auto issue = [&](uint32_t base, uint32_t h) {
+    const uint32_t i = base + (uint32_t)lane;
+    const bool a = (uint32_t)lane < depth && i < calls;
+    uint8_t* dst = smem + ((size_t)h * depth + (a ? lane : 0)) * chunk;
+    if (!raw) {
+      tk = gread_lanes_issue(c, a ? fd : -1, a ? my[i] : 0, a ? chunk : 0, dst);
+    } else {
+      const uint32_t n = min(depth, calls - base);
+      if (lane == 0) {
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        detail::mbar_expect_tx(&raw_mbar, n * chunk);
+      }
+      __syncwarp();
+      if (a) detail::tma_load(dst, rawp + my[i], chunk, &raw_mbar);
+    }
+  };
+  auto wait = [&]() {
+    if (!raw) {
+      const int64_t r = gread_lanes_wait(c, tk);
+      if (r < 0) note_err(err, r);
+    } else {
+      detail::mbar_wait(&raw_mbar, raw_ph);
+      raw_ph ^= 1u;
+    }
+  };
+  if (wid == 0) issue(0, 0);
+  uint64_t s = 0;
+  for (uint32_t base = 0, h = 0; base < calls; base += depth, h ^= 1u) {
+    if (wid == 0) wait();  // half h holds calls [base, base + depth)
+    __syncthreads();
+    if (wid == 0 && base + depth < calls) issue(base + depth, h ^ 1u);
+    const uint32_t n = min(depth, calls - base);
+    for (uint32_t q = 0; q < n; ++q)
+      s += checksum_words(smem + ((size_t)h * depth + q) * chunk, my[base + q], chunk, tid, nthr, false);
+    __syncthreads();  // half h is free for the issue two rounds on
+  }
+  s = warp_sum(s);
+  if (lane == 0) atomicAdd((unsigned long long*)sum, (unsigned long long)s);
+  if (!raw) gclose(c, fd);
+}
+
 __global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
                                const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret,
                                int flags) {
@@ -520,6 +589,24 @@ GFS_API int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path,
   if (smem > 48 * 1024) cudaFuncSetAttribute(k_randread_warp, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   k_randread_warp<<<grid, block, smem, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk,
                                              calls_per_block, d_off, d_sum, d_err);
+  return launch_err(cudaGetLastError());
+}
+
+GFS_API int gfs_run_randread_async(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
+                                   uint32_t chunk, uint32_t calls_per_block, uint32_t depth, const uint64_t* d_off,
+                                   uint64_t* d_sum, int64_t* d_err, uint32_t grid, uint32_t block) {
+  if ((!raw && !h) || (raw && !d_raw) || grid == 0 || block < 32 || block > 256 || (block & 31) || chunk == 0 ||
+      (chunk & 15) || depth == 0 || depth > 32 || (uint64_t)chunk * depth * 2 > 200 * 1024)
+    return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  gfs_launch::ArgStage as(raw ? nullptr : h, s);
+  if (!raw)
+    if (const int e = as.stage(&path, 1)) return e;
+  const char* dp = raw ? nullptr : as.str(0);
+  const uint32_t smem = chunk * depth * 2;
+  if (smem > 48 * 1024) cudaFuncSetAttribute(k_randread_async, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  k_randread_async<<<grid, block, smem, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk,
+                                              calls_per_block, depth, d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
 
