@@ -381,8 +381,7 @@ def c2_phase(X):
     if not args.no_zc:
         try:
             t0 = time.perf_counter()
-            for p_ in paths:
-                fs.register_file(p_)
+            modes = [fs.register_file(p_) for p_ in paths]
             reg_s = time.perf_counter() - t0
             fs.stats(reset=True)
             zt = []
@@ -396,6 +395,7 @@ def c2_phase(X):
             m, sd = mstd(zt)
             res["zero_copy"] = {"GBps": round(gbs(size, m), 3), "stddev": round(gbs(size, m) * sd / m, 3),
                                 "frac_h2d": round(gbs(size, m) / h2d, 4), "register_s": round(reg_s, 2),
+                                "registered_read_only": all(x == 1 for x in modes),
                                 "zc_fill": zst["zc_fill"], "rpc_read": zst["rpc_read"],
                                 "path_used": zst["zc_fill"] > 0 and zst["rpc_read"] == 0,
                                 "parity": all(sums.get("zc", [False]))}

@@ -114,15 +114,18 @@ int gfs_export(gfs_handle* h, gfs_export_desc* out);
  * barrier). */
 int gfs_attach_peer(gfs_handle* h, const gfs_export_desc* d);
 
-/* Zero-copy misses: map `path` (an existing, non-empty file; opened
- * read-write so its shared mapping can be registered) into the GPU's address
- * space with cudaHostRegister. Later O_RDONLY opens of the same file (same
+/* Zero-copy misses: map `path` (an existing, non-empty file) into the GPU's
+ * address space with cudaHostRegister: first a read-only shared mapping
+ * registered read-only (cudaHostRegisterReadOnly: the file may be read-only to
+ * the caller, and no device store can reach it); if the driver refuses that,
+ * a read-write shared mapping. Later O_RDONLY opens of the same file (same
  * st_dev, st_ino and size) fill their misses by pulling the page straight
  * from the host page cache over PCIe: no READ RPC, no staging slot, no daemon
  * memcpy. A setup call (seconds per tens of GiB); the mapping lives until
  * gfs_shutdown. The file must not change size or be replaced while
- * registered (weak consistency as for any open file, R4). -errno on failure
- * (-EIO if CUDA refuses the registration). */
+ * registered (weak consistency as for any open file, R4). Returns 1 (read-only
+ * registration) or 0 (read-write), -errno on failure (-EIO if CUDA refuses
+ * the registration). */
 int gfs_register_file(gfs_handle* h, const char* path);
 
 /* Copy the device counters (GFS_C_*, summed over shards) into out[0..n). */

@@ -437,7 +437,11 @@ __device__ int32_t rpc_complete(const gfs_ctx* c, uint64_t t, gfs_rpc_resp* resp
     backoff(ns);
     if (timed_out(c, t0)) {
       ctr(c, GFS_C_TIMEOUT);
-      return -ETIMEDOUT;  // slot is not released: the daemon is gone
+      // release the slot anyway: the ticket's successor waits for this ack, and
+      // a late completion of this ticket carries its own sequence number (the
+      // successor waits for t + R + 1), so it cannot be taken for the next one
+      st_rel64(&c->ack[slot], (uint64_t)(t + 1));
+      return -ETIMEDOUT;
     }
   }
   const int32_t res = (int32_t)(uint32_t)(v & 0xFFFFFFFFull);
@@ -779,7 +783,11 @@ __device__ __forceinline__ void pristine_free(const gfs_ctx* c, uint32_t f) {
 
 // Write back a frame's dirty range from one thread (the caller owns the frame:
 // EVICTING, ref 0): copy it into a staging slot over PCIe, then WRITE RPC.
-__device__ __noinline__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t hfid) {
+// nowait: if the staging slots it needs are not free right now, return
+// -EAGAIN instead of waiting (eviction: the caller may hold a staging slot of
+// its own, so waiting here would be hold-and-wait; it picks another victim).
+__device__ __noinline__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t f, uint32_t hfid,
+                                                     bool nowait = false) {
   const uint32_t lo = ld_rlx(&c->f_lo[f]);
   if (lo == GFS_DIRTY_NONE) return 0;
   const uint32_t hi = ld_rlx(&c->f_hi[f]);
@@ -799,6 +807,7 @@ __device__ __noinline__ int32_t frame_writeback_lane(const gfs_ctx* c, uint32_t 
       }
     }
     if (st >= 0) break;
+    if (nowait) return -EAGAIN;
     backoff(ns);
     if (timed_out(c, t0)) return -ETIMEDOUT;
   }
@@ -899,8 +908,8 @@ __device__ __noinline__ int alloc_frame(const gfs_ctx* c, uint64_t tag, uint32_t
       const uint32_t f = (uint32_t)best;
       if (ld_rlx(&c->f_lo[f]) != GFS_DIRTY_NONE) {
         const uint32_t fi = ld_rlx(&c->f_file[f]);
-        const int32_t r = frame_writeback_lane(c, f, ld_rlx(&c->files[fi].hfid));
-        if (r < 0) {  // keep the dirty page, try another victim
+        const int32_t r = frame_writeback_lane(c, f, ld_rlx(&c->files[fi].hfid), true);
+        if (r < 0) {  // keep the dirty page, try another victim (no free staging slot: never wait here)
           a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
           continue;
         }
@@ -2857,8 +2866,14 @@ __device__ inline int gmsync(const gfs_ctx* c, void* addr, uint64_t len, int fla
   return (int)sc.ret;
 }
 
-// gftruncate: host ftruncate and reclaim cached pages beyond the new size
-// (Tab.1; used by the mat-vec output).
+// gftruncate: reclaim the cached pages beyond the new size, clip the page the
+// new EOF falls in, then ftruncate on the host (Tab.1; used by the
+// mat-vec output). Pages past EOF are dropped (their dirty bytes are
+// past the end of the file: discarding them is the truncate); the boundary
+// page keeps only [0, size % P) — its dirty range is clipped and its tail
+// zeroed — so no later write-back can grow the file again. Returns 0, or
+// -EBUSY (nothing truncated on the host) if a page to drop or clip is mapped
+// or in use: the caller coordinates truncation with its readers (Tab.1).
 __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
   using namespace detail;
   Scratch& sc = scratch();
@@ -2866,14 +2881,13 @@ __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
   __syncthreads();
   if (tid == 0) {
     FileSnap s;
+    sc.frame[0] = -1;
     if (!snap_fd(c, fd, &s) || !(s.oflags & GFS_O_WRITABLE)) {
       sc.ret = -EBADF;
     } else {
       sc.fs = s;
       sc.err = 0;
-      const int32_t r = rpc_call(c, GFS_OP_TRUNC, s.hfid, 0, -1, 0, 0, size, nullptr, 0, nullptr);
-      sc.ret = r < 0 ? r : 0;
-      if (r >= 0) st_rlx64((uint64_t*)&c->files[fd].size, size);
+      sc.ret = 0;
     }
   }
   __syncthreads();
@@ -2885,6 +2899,52 @@ __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
   if (np > first) {
     const int r = drop_pages(c, fs, first, np, tid, nthr);
     if (r < 0) atomicMin(&sc.err, r);
+  }
+  const uint32_t keep = (uint32_t)(size & (P - 1));
+  if (tid == 0 && keep && (size >> c->page_shift) < np) {  // the page the new EOF falls in
+    const uint64_t b = size >> c->page_shift;
+    uint64_t* slot = walk(c, fs.root, fs.height, b, false, nullptr);
+    const uint64_t sv = slot ? ld_acq64(slot) : 0;
+    if ((uint32_t)sv) {
+      const uint32_t f = (uint32_t)sv - 1u;
+      const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)b;
+      if (ld_acq64(&c->f_tag[f]) == want) {
+        if (!claim_frame(&c->f_state[f], 0u)) {
+          atomicMin(&sc.err, -EBUSY);
+        } else if (ld_acq64(&c->f_tag[f]) != want) {
+          a64_and_rel(&c->f_state[f], fl64(GFS_ST_EVICTING));
+        } else {
+          const uint32_t lo = ld_rlx(&c->f_lo[f]);
+          if (lo != GFS_DIRTY_NONE) {
+            const uint32_t hi = ld_rlx(&c->f_hi[f]);
+            if (lo >= keep) {  // every dirty byte is past the new EOF
+              st_rlx(&c->f_lo[f], GFS_DIRTY_NONE);
+              st_rlx(&c->f_hi[f], 0);
+              st_rlx(&c->f_written[f], 0);
+            } else if (hi > keep) {
+              st_rlx(&c->f_hi[f], keep);
+              const uint32_t wr = ld_rlx(&c->f_written[f]);
+              if (wr > keep - lo) st_rlx(&c->f_written[f], keep - lo);
+            }
+          }
+          if (ld_rlx(&c->f_valid[f]) > keep) st_rlx(&c->f_valid[f], keep);
+          if (ld_rlx(&c->f_hv[f]) > keep) st_rlx(&c->f_hv[f], keep);
+          sc.frame[0] = (int)f;  // the block zeroes its tail, then it is released
+        }
+      }
+    }
+  }
+  __syncthreads();
+  if (sc.frame[0] >= 0) {
+    block_zero(frame_ptr(c, (uint32_t)sc.frame[0]) + keep, P - keep, tid, nthr);
+    __threadfence();
+    __syncthreads();
+    if (tid == 0) a64_and_rel(&c->f_state[(uint32_t)sc.frame[0]], fl64(GFS_ST_EVICTING));
+  }
+  if (tid == 0 && sc.err == 0) {  // nothing cached can reach past `size` any more: truncate the host file
+    const int32_t r = rpc_call(c, GFS_OP_TRUNC, fs.hfid, 0, -1, 0, 0, size, nullptr, 0, nullptr);
+    if (r < 0) sc.err = r;
+    else st_rlx64((uint64_t*)&c->files[fd].size, size);
   }
   __syncthreads();
   return sc.err;

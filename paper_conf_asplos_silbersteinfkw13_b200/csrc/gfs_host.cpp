@@ -251,6 +251,7 @@ struct gfs_handle {
     uint8_t* map;
     uint64_t dptr;
     int fd;
+    bool ro;                     // read-only mapping registered read-only
   };
   SpinMutex zc_mu;
   std::vector<ZcFile> zc;
@@ -1236,33 +1237,51 @@ GFS_API int gfs_attach_peer(gfs_handle* h, const gfs_export_desc* d) {
 
 GFS_API int gfs_register_file(gfs_handle* h, const char* path) {
   if (!h || !path) return -EINVAL;
-  const int fd = ::open(path, O_RDWR);  // a read-only mapping cannot be registered (measured: invalid argument)
-  if (fd < 0) return -errno;
-  struct stat st;
-  if (fstat(fd, &st) != 0 || st.st_size <= 0) {
-    const int e = st.st_size <= 0 ? -EINVAL : -errno;
-    ::close(fd);
-    return e;
-  }
-  const uint64_t size = (uint64_t)st.st_size;
-  void* m = mmap(nullptr, size, PROT_READ | PROT_WRITE, MAP_SHARED, fd, 0);
-  if (m == MAP_FAILED) {
-    const int e = -errno;
-    ::close(fd);
-    return e;
-  }
   cudaSetDevice(h->cfg.device);
-  void* d = nullptr;
-  if (cudaHostRegister(m, size, cudaHostRegisterMapped) != cudaSuccess ||
-      cudaHostGetDevicePointer(&d, m, 0) != cudaSuccess) {
-    fprintf(stderr, "gpufs: cudaHostRegister(%s): %s\n", path, cudaGetErrorString(cudaGetLastError()));
-    munmap(m, size);
-    ::close(fd);
-    return -EIO;
+  // First a read-only registration of a read-only mapping (the GPU only pulls
+  // from it; an input the caller cannot write can be registered, and no
+  // device store can reach the file). Drivers that refuse to register a
+  // PROT_READ mapping get the read-write mapping instead (measured in round 1
+  // on this image: cudaHostRegister of a PROT_READ mapping -> invalid argument).
+  for (int attempt = 0; attempt < 2; ++attempt) {
+    const bool ro = attempt == 0;
+    const int fd = ::open(path, ro ? O_RDONLY : O_RDWR);
+    if (fd < 0) {
+      if (ro) continue;
+      return -errno;
+    }
+    struct stat st;
+    if (fstat(fd, &st) != 0) {
+      const int e = -errno;
+      ::close(fd);
+      return e;
+    }
+    if (st.st_size <= 0) {
+      ::close(fd);
+      return -EINVAL;
+    }
+    const uint64_t size = (uint64_t)st.st_size;
+    void* m = mmap(nullptr, size, ro ? PROT_READ : (PROT_READ | PROT_WRITE), MAP_SHARED, fd, 0);
+    if (m == MAP_FAILED) {
+      const int e = -errno;
+      ::close(fd);
+      return e;
+    }
+    void* d = nullptr;
+    const unsigned flags = cudaHostRegisterMapped | (ro ? cudaHostRegisterReadOnly : 0u);
+    if (cudaHostRegister(m, size, flags) != cudaSuccess || cudaHostGetDevicePointer(&d, m, 0) != cudaSuccess) {
+      const cudaError_t e = cudaGetLastError();  // clears the error for the next attempt
+      munmap(m, size);
+      ::close(fd);
+      if (ro) continue;
+      fprintf(stderr, "gpufs: cudaHostRegister(%s): %s\n", path, cudaGetErrorString(e));
+      return -EIO;
+    }
+    std::lock_guard<SpinMutex> g(h->zc_mu);
+    h->zc.push_back({(uint64_t)st.st_dev, (uint64_t)st.st_ino, size, (uint8_t*)m, (uint64_t)(uintptr_t)d, fd, ro});
+    return ro ? 1 : 0;
   }
-  std::lock_guard<SpinMutex> g(h->zc_mu);
-  h->zc.push_back({(uint64_t)st.st_dev, (uint64_t)st.st_ino, size, (uint8_t*)m, (uint64_t)(uintptr_t)d, fd});
-  return 0;
+  return -EIO;
 }
 
 GFS_API int gfs_stats(gfs_handle* h, uint64_t* out, int n, int reset) {

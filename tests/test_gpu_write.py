@@ -133,6 +133,31 @@ def test_gftruncate(g, shmdir):
     assert host(path) == b"abc"
 
 
+def test_gftruncate_unaligned_clips_the_boundary_page(g, shmdir):
+    """Truncate a write-once file held open (its pages dirty in the cache) to a size
+    that is not page-aligned: the page the new EOF falls in keeps only its bytes
+    below EOF (a later write-back must not grow the file again), the
+    pages past it are dropped, and bytes written later past the old EOF leave
+    zeros in between (P:L321-324)."""
+    P = 4096
+    path = os.path.join(shmdir, "tu.bin")
+    data = rnd(3 * P + 100, 7)
+    cut = P + 1000
+    with g.GpuFS(cache_bytes=64 * P, page_size=P, timeout_ms=30000, daemon_threads=2) as fs:
+        fd = fs.pin(path, flags=1)  # held open across the launches: the dirty pages stay this incarnation's
+        assert fd >= 0
+        assert (fs.gwrite_calls(path, [0], [len(data)], data) == len(data)).all()
+        assert fs.gftruncate(path, cut) == 0
+        assert os.path.getsize(path) == cut
+        assert fs.gfstat(path, flags=1) == cut
+        assert fs.gfsync(path) == 0
+        assert host(path) == data[:cut]  # the clipped page wrote back [0, cut % P) only
+        fs.gwrite_calls(path, [2 * P], [10], b"z" * 10)
+        assert fs.gfsync(path) == 0
+        assert fs.unpin(fd) == 0
+    assert host(path) == data[:cut] + bytes(2 * P - cut) + b"z" * 10
+
+
 def test_more_files_than_fd_cache(g, shmdir):
     """The daemon's fd cache closes idle host fds and re-opens them by path."""
     paths = []
