@@ -652,18 +652,18 @@ def matvec_phase(X, h2d):
 
 
 # ---------------------------------------------------------------------- grep (C1, C4)
-def grep_run(X, fs, d, lst, reps, hits, file_ids, chunk=32768):
+def grep_run(X, fs, d, lst, reps, hits, file_ids, chunk=16384, block=128):
     """cold (first run on fs) + warm runs (files kept open): device ms of each."""
     torch = X.torch
     state = fs.grep_state(d, lst, hits=hits, keep_open=True, rec_cap=1 << 24, pair_cap=1 << 23, chunk=chunk,
-                          file_ids=file_ids)
+                          block=block, file_ids=file_ids)
     times = []
     for it in range(1 + reps):
         X.barrier()
         t = X.timed(lambda: fs.grep(d, lst, hits=hits, keep_open=True, stream=X.stream, sync=False, state=state,
-                                    chunk=chunk), 1)
+                                    chunk=chunk, block=block), 1)
         times += t
-    out = fs.grep(d, lst, hits=hits, keep_open=True, stream=X.stream, state=state, chunk=chunk)
+    out = fs.grep(d, lst, hits=hits, keep_open=True, stream=X.stream, state=state, chunk=chunk, block=block)
     return times[0], times[1:], out
 
 

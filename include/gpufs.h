@@ -273,6 +273,13 @@ typedef struct gfs_grep_params {
                            records, hits and the digest (e.g. a shard's global indices); NULL:
                            the list index i */
   uint64_t rec_cap;     /* records the work area can stage (>= the records found, else -ENOSPC) */
+  uint32_t whole_max;   /* a file of more than one chunk and at most this many bytes is ONE work
+                           item: one block scans it chunk after chunk, counting in shared memory,
+                           and emits its records directly (0: 64 bytes per count-table slot, the
+                           slots being what shared memory allows at >= 768 threads per SM:
+                           4096 at block 256 / chunk 16 KiB, 1024 at block 128; <= chunk: never). Larger
+                           files are split into chunk items merged through the (file, word) table */
+  uint32_t pad0;
 } gfs_grep_params;
 
 /* Device scratch bytes gfs_grep needs for these parameters. */

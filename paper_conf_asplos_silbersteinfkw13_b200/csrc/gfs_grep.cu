@@ -15,9 +15,10 @@
 //                 list), record each line's offset;
 //   k_grep_open   one warp per file builds its path from the list line, gopen
 //                 (the first gopen goes to the host), gfstat;
-//   k_grep_plan   exclusive scan of per-file work-item counts; k_grep_items
-//                 writes one 32-byte descriptor per item (a whole file when it
-//                 fits one item, else a chunk of it): one round trip per item;
+//   k_grep_items  one 32-byte descriptor per work item: a file of one chunk,
+//                 a file of up to `whole_max` bytes scanned chunk after chunk
+//                 by one block (these first, most chunks first), or one chunk
+//                 of a larger file: one round trip per item;
 //   k_grep_scan   persistent blocks pull items. gread brings the item plus a
 //                 halo into shared memory (TMA). Pass 1 classifies 32-byte
 //                 stripes into word-byte bit masks (SWAR, 4 bytes per op); pass
@@ -27,8 +28,8 @@
 //                 32-byte compare on a fingerprint match. Counts per item in
 //                 shared memory; a whole-file item emits its (file, word,
 //                 count) records directly (into a record page the block
-//                 reserved), chunks of large files merge through a global
-//                 (file, word) table;
+//                 reserved), chunks of files above `whole_max` merge through
+//                 a global (file, word) table;
 //   k_grep_close  gclose every file (unless kept open for warm re-runs);
 //   k_grep_compact emit the merged records and their word totals, and leave
 //                 the (file, word) table empty for the next run;
@@ -63,7 +64,7 @@ constexpr uint64_t kPairEmpty = ~0ull;
 constexpr uint64_t kDupBit = 1ull << 63;  // table entry: the word has duplicates
 constexpr uint64_t kKeepMagic = 0x31504545504b5247ull;  // GRKPEEP1: the persistent words are initialised
 constexpr uint64_t kPairsClean = 0x4e41454c43524150ull;  // PAIRCLEAN: the (file, word) table is empty
-constexpr uint32_t kRecPage = 2048;  // records per output page
+constexpr uint32_t kRecPage = 4096;  // records per output page (>= the count table: one item's records fit)
 constexpr uint32_t kNoPage = 0xFFFFFFFFu;
 
 // One work item (a whole file, or a chunk of a large one), precomputed by
@@ -73,10 +74,12 @@ struct ItemDesc {
   uint32_t f;       // list index
   int32_t fd;
   uint32_t gid;     // reported file id
-  uint32_t rlen;    // bytes to read (chunk + halos, clipped at EOF)
-  uint32_t body;    // bytes whose token starts this item counts (the chunk)
-  uint32_t meta;    // bit 31: a whole file (records emitted directly); bits 0..4: pre (bytes before the chunk)
+  uint32_t rlen;    // bytes to read (chunk + halos, clipped at EOF); a multi-chunk whole file: its size
+  uint32_t body;    // bytes whose token starts this item counts (the chunk); multi-chunk: the chunk count
+  uint32_t meta;    // bit 31: a whole file (records emitted directly); bit 30: multi-chunk whole file;
+                    // bits 0..4: pre (bytes before the chunk)
 };
+constexpr uint32_t kMaxWholeChunks = 31;  // chunks of a file one block scans whole (histogram buckets)
 
 struct GrepWork {
   // dictionary
@@ -85,6 +88,8 @@ struct GrepWork {
   uint32_t table_mask;
   uint32_t* dup_head;     // per primary word: first duplicate + 1
   uint32_t* dup_next;     // per word: next duplicate + 1
+  uint32_t* filt;         // one bit per filter_index() value of the words' hashes (L1-resident)
+  uint32_t filt_log2;     // log2 of the filter's bits
   // file list
   uint8_t* list;          // list_cap bytes
   uint32_t* list_chunk;   // per list chunk: line starts (then exclusive prefix)
@@ -92,10 +97,11 @@ struct GrepWork {
   const uint32_t* file_ids;  // per file: the id used in records, hits and the digest (NULL: the list index)
   int32_t* fd;
   uint64_t* size;
-  uint64_t* item_base;    // per file: first item (max_files + 1)
   struct ItemDesc* desc;  // item -> what to read and where it goes (k_grep_items)
   uint64_t max_items;
-  uint32_t chunk;         // item bytes; also the batch size in batch space
+  uint32_t chunk;         // item bytes
+  uint32_t whole_chunks;  // a file of 2..whole_chunks chunks is one item, scanned whole by one block
+  uint32_t cslots;        // count table slots per scan block (power of two)
   // (file, word) -> count table
   uint64_t* pair;         // slot i: pair[2i] = (file << 32) | word (or empty), pair[2i+1] = count
   uint64_t pair_mask;
@@ -113,7 +119,13 @@ struct GrepWork {
   unsigned long long* prof;  // GFS_GREP_PROF=1: per-phase clock cycles of the scan's thread 0 (else null)
 };
 enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS, V_DSUM, V_DXOR, V_NLISTED,
-       V_NEXTF, V_LISTSZ, V_HOLD_DICT, V_HOLD_LIST, V_NBATCH, V_NPAGES, V_PAIRS_DIRTY, V_NVARS };
+       V_NEXTF, V_LISTSZ, V_HOLD_DICT, V_HOLD_LIST, V_NPAGES, V_PAIRS_DIRTY,
+       V_NCHUNKED,                         // items of files split into chunks
+       V_CUR_CHUNKED,                      // their placement cursor (k_grep_items)
+       V_CUR_ONE,                          // one-chunk files: placement cursor = their count
+       V_WHOLE_HIST,                       // [n]: multi-chunk whole files of n chunks
+       V_WHOLE_CUR = V_WHOLE_HIST + kMaxWholeChunks + 1,  // [n]: their placement cursors
+       V_NVARS = V_WHOLE_CUR + kMaxWholeChunks + 1 };
 enum { K_MAGIC = 0, K_PAIRS, K_DICT_FD, K_LIST_FD, K_NKEEP };
 
 __device__ __forceinline__ bool is_word(uint32_t ch) {
@@ -189,6 +201,19 @@ __device__ __forceinline__ uint64_t entry_key(uint64_t h, uint32_t len) {
 }
 __device__ __forceinline__ uint64_t key_bits(uint64_t e) { return (e & ~kDupBit) >> 26; }
 
+// Pre-filter: a token whose hash has no dictionary word's bit set is not a
+// word (no false negatives; ~1 in 5 non-words pass at 4.5 bits per word). The
+// bitmap (<= 32 KiB) is read with an L1 evict_last hint: it stays in L1, so
+// most non-words end without an L2 round trip.
+__device__ __forceinline__ uint32_t filter_index(uint64_t h, uint32_t log2) {
+  return (((uint32_t)(h >> 32) ^ (uint32_t)h) * 0x9E3779B1u) >> (32 - log2);
+}
+__device__ __forceinline__ uint32_t ld_filter(const uint32_t* p) {
+  uint32_t v;
+  asm("ld.global.nc.L1::evict_last.u32 %0, [%1];" : "=r"(v) : "l"(p));
+  return v;
+}
+
 __device__ __forceinline__ uint64_t splitmix64(uint64_t x) {
   uint64_t z = x + 0x9E3779B97F4A7C15ull;
   z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
@@ -255,6 +280,7 @@ __global__ void k_grep_init(const __grid_constant__ GrepWork w, uint32_t max_wor
   const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
   const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
   for (uint64_t i = t; i <= w.table_mask; i += stride) w.table[i] = 0;
+  for (uint64_t i = t; i < (1ull << w.filt_log2) / 32; i += stride) w.filt[i] = 0;
   for (uint64_t i = t; i < max_words; i += stride) {
     w.dup_head[i] = 0;
     w.dup_next[i] = 0;
@@ -320,6 +346,8 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, const __gri
         *(uint4*)(s + 16) = q1;
         const uint64_t h = tok_hash(q0.x, q0.y, n);
         const uint64_t ent = entry_key(h, n) | (k + 1);
+        const uint32_t fi = filter_index(h, w.filt_log2);
+        atomicOr(&w.filt[fi >> 5], 1u << (fi & 31));
         // linear probing from the start of the hash's 4-entry (32-byte) bucket:
         // lookups read a whole bucket per step (probe_bucket)
         uint32_t slot = (uint32_t)h & w.table_mask & ~3u;
@@ -458,8 +486,10 @@ __global__ void k_grep_list_emit(const __grid_constant__ GrepWork w, uint32_t ma
 // --------------------------------------------------------------- open files
 // One warp per file: the path is the list line (relative lines are resolved
 // against the list's directory, R15), assembled in shared memory,
-// then gopen + gfstat. Records the file's item count and batch-space weight.
+// then gopen + gfstat. Counts the file's items: the histogram of multi-chunk
+// whole files by chunk count, the chunks of larger files.
 __device__ __forceinline__ uint64_t item_count(uint64_t size, uint32_t chunk) { return (size + chunk - 1) / chunk; }
+__device__ __forceinline__ bool whole_multi(const GrepWork& w, uint64_t nch) { return nch >= 2 && nch <= w.whole_chunks; }
 __global__ void __launch_bounds__(32) k_grep_open(const gfs_ctx* c, const __grid_constant__ GrepWork w, const char* dir, uint32_t dir_len,
                                                   uint32_t max_files) {
   __shared__ __align__(16) char pbuf[kMaxPath + 32];
@@ -511,10 +541,11 @@ __global__ void __launch_bounds__(32) k_grep_open(const gfs_ctx* c, const __grid
       if (sz < 0) {
         set_err(w, sz);
         w.size[f] = 0;
-        w.item_base[f] = 0;
       } else {
         w.size[f] = (uint64_t)sz;
-        w.item_base[f] = item_count((uint64_t)sz, w.chunk);  // counts; scanned by k_grep_plan
+        const uint64_t nch = item_count((uint64_t)sz, w.chunk);
+        if (whole_multi(w, nch)) atomicAdd(&w.vars[V_WHOLE_HIST + nch], 1ull);
+        else if (nch > 1) atomicAdd(&w.vars[V_NCHUNKED], (unsigned long long)nch);
         atomicAdd(&w.vars[V_BYTES], (unsigned long long)sz);
       }
     }
@@ -522,91 +553,110 @@ __global__ void __launch_bounds__(32) k_grep_open(const gfs_ctx* c, const __grid
   }
 }
 
-// --------------------------------------------------------------- plan
-// One block: exclusive scan of the per-file item counts (item_base), in
-// tiles of 4 * blockDim counts (each thread 4 consecutive ones), the tile's
-// loads issued before the previous tile's scan is used.
-__global__ void k_grep_plan(const __grid_constant__ GrepWork w) {
-  __shared__ uint64_t wsum[32];
-  __shared__ uint64_t carry_s;
-  const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31, wid = tid >> 5, nw = nthr >> 5;
-  const uint64_t n = w.vars[V_NFILES];
-  const uint64_t tile = 4ull * nthr;
-  if (tid == 0) carry_s = 0;
-  __syncthreads();
-  for (uint64_t t0 = 0; t0 < n; t0 += tile) {
-    uint64_t v[4];
-    uint64_t mine = 0;
-#pragma unroll
-    for (int q = 0; q < 4; ++q) {
-      const uint64_t i = t0 + 4ull * tid + q;
-      v[q] = i < n ? w.item_base[i] : 0;
-      mine += v[q];
-    }
-    uint64_t incl = mine;
-    for (int o = 1; o < 32; o <<= 1) {
-      const uint64_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
-      if (lane >= o) incl += t;
-    }
-    if (lane == 31) wsum[wid] = incl;
-    __syncthreads();
-    uint64_t base = carry_s + incl - mine, all = 0;
-    for (int q = 0; q < nw; ++q) {
-      base += q < wid ? wsum[q] : 0;
-      all += wsum[q];
-    }
-#pragma unroll
-    for (int q = 0; q < 4; ++q) {
-      const uint64_t i = t0 + 4ull * tid + q;
-      if (i < n) w.item_base[i] = base;
-      base += v[q];
-    }
-    __syncthreads();
-    if (tid == 0) carry_s += all;
-    __syncthreads();
-  }
+// --------------------------------------------------------------- items
+// Item order: the multi-chunk whole files first, most chunks first (the
+// longest items start first: no block is left with a long item at the end),
+// then the chunks of larger files, then the one-chunk files. Positions come
+// from cursors: per chunk count for the whole files (one atomic per group of
+// equal counts in a warp), one per block for the rest (block scan). Order
+// within a class is arbitrary; the results do not depend on it.
+__global__ void __launch_bounds__(256) k_grep_items(const __grid_constant__ GrepWork w) {
+  __shared__ unsigned long long base_s[kMaxWholeChunks + 2];  // [n]: first item of n-chunk whole files
+  __shared__ unsigned long long blk_s[2];
+  __shared__ uint32_t wsum[2][8];
+  const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
+  const uint32_t n = (uint32_t)w.vars[V_NFILES];
   if (tid == 0) {
-    uint64_t r0 = carry_s;
-    if (r0 > w.max_items) {
-      set_err(w, -ENOSPC);
-      r0 = w.max_items;
+    unsigned long long o = 0;
+    for (uint32_t k = kMaxWholeChunks; k >= 2; --k) {
+      base_s[k] = o;
+      o += w.vars[V_WHOLE_HIST + k];
     }
-    w.vars[V_NITEMS] = r0;
-    w.item_base[n] = r0;
+    base_s[kMaxWholeChunks + 1] = o;  // = whole multi-chunk items; chunked items follow
+    blk_s[0] = o;
+    blk_s[1] = o + w.vars[V_NCHUNKED];  // one-chunk files follow the chunked ones
+  }
+  __syncthreads();
+  const unsigned long long nwhole = blk_s[0], chunk_end = blk_s[1];
+  for (uint32_t f0 = blockIdx.x * 256u; f0 < n; f0 += gridDim.x * 256u) {
+    const uint32_t f = f0 + tid;
+    const bool valid = f < n;
+    const uint64_t size = valid ? w.size[f] : 0;
+    const uint64_t nch = item_count(size, w.chunk);
+    const bool multi = valid && whole_multi(w, nch);
+    const uint32_t u_chunks = (valid && !multi && nch > 1) ? (uint32_t)nch : 0u;
+    const uint32_t u_one = (valid && nch == 1) ? 1u : 0u;
+    // block scan of both counts
+    uint32_t a = u_chunks, b = u_one;
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t ta = __shfl_up_sync(0xFFFFFFFFu, a, o), tb = __shfl_up_sync(0xFFFFFFFFu, b, o);
+      if (lane >= o) {
+        a += ta;
+        b += tb;
+      }
+    }
+    if (lane == 31) {
+      wsum[0][wid] = a;
+      wsum[1][wid] = b;
+    }
+    __syncthreads();
+    uint32_t oa = a - u_chunks, ob = b - u_one, ta = 0, tb = 0;
+    for (int q = 0; q < 8; ++q) {
+      oa += q < wid ? wsum[0][q] : 0u;
+      ob += q < wid ? wsum[1][q] : 0u;
+      ta += wsum[0][q];
+      tb += wsum[1][q];
+    }
+    if (tid == 0) {
+      blk_s[0] = ta ? atomicAdd(&w.vars[V_CUR_CHUNKED], (unsigned long long)ta) : 0;
+      blk_s[1] = tb ? atomicAdd(&w.vars[V_CUR_ONE], (unsigned long long)tb) : 0;
+    }
+    // whole multi-chunk files: one atomic per group of equal chunk counts
+    const uint32_t key = multi ? (uint32_t)nch : 0xFFFFFFFFu;
+    const uint32_t peers = __match_any_sync(0xFFFFFFFFu, key);
+    unsigned long long wpos = 0;
+    if (multi) {
+      const int leader = __ffs(peers) - 1;
+      unsigned long long b0 = 0;
+      if (lane == leader) b0 = atomicAdd(&w.vars[V_WHOLE_CUR + nch], (unsigned long long)__popc(peers));
+      b0 = __shfl_sync(peers, b0, leader);
+      wpos = base_s[nch] + b0 + __popc(peers & ((1u << lane) - 1u));
+    }
+    __syncthreads();
+    if (valid && nch) {
+      ItemDesc d;
+      d.f = f;
+      d.fd = w.fd[f];
+      d.gid = gid_of(w, f);
+      if (nch == 1 || multi) {  // a whole file
+        d.roff = 0;
+        d.rlen = (uint32_t)size;
+        d.body = multi ? (uint32_t)nch : (uint32_t)size;
+        d.meta = multi ? (3u << 30) : (1u << 31);
+        const unsigned long long pos = multi ? wpos : chunk_end + blk_s[1] + ob;
+        if (pos < w.max_items) w.desc[pos] = d;
+      } else {  // chunk [s, e) with up to kPre bytes before and kHalo after
+        const unsigned long long p0 = nwhole + blk_s[0] + oa;
+        for (uint64_t i = 0; i < nch; ++i) {
+          const uint64_t s = i * w.chunk, e = min(size, s + w.chunk);
+          const uint64_t ws = s >= kPre ? s - kPre : 0, we = min(size, e + kHalo);
+          d.roff = ws;
+          d.rlen = (uint32_t)(we - ws);
+          d.body = (uint32_t)(e - s);
+          d.meta = (uint32_t)(s - ws);
+          if (p0 + i < w.max_items) w.desc[p0 + i] = d;
+        }
+      }
+    }
+    __syncthreads();  // blk_s and wsum are reused
   }
 }
 
-// item -> descriptor (file, batch-space offset, what to read)
-__global__ void k_grep_items(const __grid_constant__ GrepWork w) {
-  const uint32_t n = (uint32_t)w.vars[V_NFILES];
-  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-  const uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
-  for (uint64_t f = t; f < n; f += stride) {
-    const uint64_t a = w.item_base[f], b = min(w.item_base[f + 1], w.max_items);
-    const uint64_t size = w.size[f];
-    const uint32_t gid = gid_of(w, (uint32_t)f);
-    const int32_t fd = w.fd[f];
-    for (uint64_t i = a; i < b; ++i) {
-      ItemDesc d;
-      d.f = (uint32_t)f;
-      d.fd = fd;
-      d.gid = gid;
-      if (b - a == 1) {  // a whole file
-        d.roff = 0;
-        d.rlen = (uint32_t)size;
-        d.body = (uint32_t)size;
-        d.meta = 1u << 31;
-      } else {  // chunk [s, e) with up to kPre bytes before and kHalo after
-        const uint64_t s = (i - a) * w.chunk, e = min(size, s + w.chunk);
-        const uint64_t ws = s >= kPre ? s - kPre : 0, we = min(size, e + kHalo);
-        d.roff = ws;
-        d.rlen = (uint32_t)(we - ws);
-        d.body = (uint32_t)(e - s);
-        d.meta = (uint32_t)(s - ws);
-      }
-      w.desc[i] = d;
-    }
-  }
+// The item count (all classes, after k_grep_items) and its bound.
+__device__ uint64_t count_items(const GrepWork& w) {
+  unsigned long long t = w.vars[V_NCHUNKED] + w.vars[V_CUR_ONE];
+  for (uint32_t k = 2; k <= kMaxWholeChunks; ++k) t += w.vars[V_WHOLE_HIST + k];
+  return t;
 }
 
 // --------------------------------------------------------------- scan
@@ -623,7 +673,10 @@ __device__ __forceinline__ uint32_t bit_range(int lo, int hi) {
 __device__ __noinline__ void pair_add(const GrepWork& w, uint32_t f, uint32_t k, uint64_t cnt) {
   const uint64_t key = ((uint64_t)f << 32) | k;
   uint64_t slot = splitmix64(key) & w.pair_mask;
-  for (uint64_t probe = 0; probe <= w.pair_mask; ++probe, slot = (slot + 1) & w.pair_mask) {
+  // a run this long means the table is (nearly) full: report it rather than
+  // walk the whole table for every add
+  const uint64_t limit = w.pair_mask < 4095 ? w.pair_mask : 4095;
+  for (uint64_t probe = 0; probe <= limit; ++probe, slot = (slot + 1) & w.pair_mask) {
     const unsigned long long cur = atomicCAS((unsigned long long*)&w.pair[2 * slot], (unsigned long long)kPairEmpty,
                                              (unsigned long long)key);
     if (cur == kPairEmpty || cur == key) {
@@ -661,14 +714,18 @@ struct ScanAcc {
   uint64_t dsum, dxor, nh;
 };
 
-constexpr uint32_t kCountSlots = 2048;
+// Count table slots per block: the distinct words of one item (a 16 KiB chunk
+// of the C4 corpus has ~450, a 256 KiB file ~3000); an item that exhausts the
+// 64-probe limit spills to the global (file, word) table (still exact)
+constexpr uint32_t kMaxCountSlots = 4096;  // (runtime: GrepWork.cslots, a power of two)
+static_assert(kRecPage >= kMaxCountSlots, "one item's records fit one record page");
 // Shared-memory state of one scan block (dynamic shared memory, see scan_smem).
 struct ScanSmem {
   uint8_t* buf;     // kPre + chunk + kHalo + kSlack bytes; file byte p at buf[kPre + p - s]
   uint32_t* mask;   // word-byte bits per 32-byte stripe of buf (+1 zero stripe)
   uint32_t* ckey;   // count table: word + 1 (0 = empty)
   uint32_t* ccnt;
-  uint16_t* olist;  // occupied count slots, in insertion order
+  uint32_t* occ;    // occupied count slots, one bit each
   uint64_t hf;      // splitmix64(file index) of the current item (digest)
   uint32_t cmask;   // count table slots - 1
 };
@@ -683,13 +740,11 @@ __device__ __forceinline__ uint32_t atoms_cas(uint32_t* p, uint32_t cmp, uint32_
                : "memory");
   return r;
 }
-__device__ __forceinline__ uint32_t atoms_add(uint32_t* p, uint32_t v) {
-  uint32_t r;
-  asm volatile("atom.shared.add.u32 %0, [%1], %2;" : "=r"(r) : "r"(detail::smem_u32(p)), "r"(v) : "memory");
-  return r;
-}
 __device__ __forceinline__ void reds_add(uint32_t* p, uint32_t v) {
   asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(detail::smem_u32(p)), "r"(v) : "memory");
+}
+__device__ __forceinline__ void reds_or(uint32_t* p, uint32_t v) {
+  asm volatile("red.shared.or.b32 [%0], %1;" ::"r"(detail::smem_u32(p)), "r"(v) : "memory");
 }
 
 // The rare per-hit paths, out of line (the token loop keeps its registers).
@@ -708,14 +763,14 @@ __device__ __noinline__ void hit_list(const GrepWork& w, uint32_t f, uint32_t k,
 
 // One hit of word k at file position pos: per-item shared count (spilling to
 // the global table when the probe run is exhausted), digest, optional hit list.
-__device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
+__device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, uint32_t* spilled,
                                           uint32_t f, uint32_t k, uint64_t pos, uint64_t* hits, uint64_t hit_cap,
                                           ScanAcc& acc) {
   uint32_t cs = (k * 2654435761u) & S.cmask;
   bool done = false;
   for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & S.cmask) {
     const uint32_t prev = atoms_cas(&S.ckey[cs], 0u, k + 1);
-    if (prev == 0) S.olist[atoms_add(nocc, 1u)] = (uint16_t)cs;
+    if (prev == 0) reds_or(&S.occ[cs >> 5], 1u << (cs & 31));
     if (prev == 0 || prev == k + 1) {
       reds_add(&S.ccnt[cs], 1u);
       done = true;
@@ -731,7 +786,7 @@ __device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, 
 }
 
 // One token: bytes buf[i, i + L), file position pos, 1 <= L <= 32.
-__device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S, uint32_t* nocc, uint32_t* spilled,
+__device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S, uint32_t* spilled,
                                            uint32_t f, uint32_t i, uint32_t L, uint64_t pos, uint64_t* hits,
                                            uint64_t hit_cap, ScanAcc& acc) {
   // first 8 bytes: three aligned words and two funnel shifts
@@ -740,6 +795,8 @@ __device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S,
   const uint32_t w0 = low_bytes(__funnelshift_r(a0, a1, r8), min((int)L, 4));
   const uint32_t w1 = low_bytes(__funnelshift_r(a1, a2, r8), min(max((int)L - 4, 0), 4));
   const uint64_t h = tok_hash(w0, w1, L);
+  const uint32_t fi = filter_index(h, w.filt_log2);
+  if (!((ld_filter(&w.filt[fi >> 5]) >> (fi & 31)) & 1u)) return;
   const uint64_t want = entry_key(h, L) >> 26;
   // One 32-byte bucket (4 entries) per step; insertion filled the first empty
   // slot in the same order, so an empty slot ends the search.
@@ -774,10 +831,10 @@ __device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S,
         const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
                            (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
         if (same) {
-          count_hit(w, S, nocc, spilled, f, kp, pos, hits, hit_cap, acc);
+          count_hit(w, S, spilled, f, kp, pos, hits, hit_cap, acc);
           if (ent[q] & kDupBit) {  // the word's duplicates each count (R14)
             for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
-              count_hit(w, S, nocc, spilled, f, d - 1, pos, hits, hit_cap, acc);
+              count_hit(w, S, spilled, f, d - 1, pos, hits, hit_cap, acc);
           }
           return;
         }
@@ -788,8 +845,36 @@ __device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S,
   }
 }
 
-// Bits [lo, hi) of a 32-bit mask (lo, hi clamped to [0, 32]).
+// The byte ranges of chunk ci of item d: token starts in [s, e) count, [ws, we)
+// is read (the chunk with up to kPre bytes before and kHalo after).
+struct StepRange {
+  uint64_t s, e, ws, we;
+};
+__device__ __forceinline__ StepRange step_range(const ItemDesc& d, uint32_t ci, uint32_t chunk) {
+  StepRange r;
+  if ((d.meta >> 30) & 1u) {  // multi-chunk whole file: rlen is its size
+    r.s = (uint64_t)ci * chunk;
+    r.e = min((uint64_t)d.rlen, r.s + chunk);
+    r.ws = r.s >= kPre ? r.s - kPre : 0;
+    r.we = min((uint64_t)d.rlen, r.e + kHalo);
+  } else if (d.meta >> 31) {  // one-chunk file
+    r.s = r.ws = 0;
+    r.e = r.we = d.rlen;
+  } else {  // a chunk of a larger file
+    r.ws = d.roff;
+    r.we = r.ws + d.rlen;
+    r.s = r.ws + (d.meta & 31u);
+    r.e = r.s + d.body;
+  }
+  return r;
+}
+__device__ __forceinline__ uint32_t item_chunks(const ItemDesc& d) { return ((d.meta >> 30) & 1u) ? d.body : 1u; }
 
+// Persistent blocks pull items; an item is one chunk of a large file, a
+// one-chunk file, or a multi-chunk file of at most whole_max bytes that the
+// block scans chunk after chunk, counting in shared memory across chunks.
+// Thread 0 claims the next item and loads its descriptor while the block
+// works on the current one (the claim and the descriptor load are off the path).
 __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __grid_constant__ GrepWork w, uint32_t chunk, uint64_t* hits,
                                                    uint64_t hit_cap, uint64_t* totals, uint32_t* rec,
                                                    uint64_t rec_cap) {
@@ -801,40 +886,39 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __
   S.buf = sm;
   S.mask = (uint32_t*)(sm + buf_bytes);
   S.ckey = S.mask + ((nstripe_max + 1 + 3) & ~3u);
-  S.ccnt = S.ckey + kCountSlots;
-  S.olist = (uint16_t*)(S.ccnt + kCountSlots);
-  S.cmask = kCountSlots - 1;
-  uint16_t* tok = S.olist + kCountSlots;  // token starts of one round: <= 32 per thread
+  const uint32_t cslots = w.cslots;
+  S.ccnt = S.ckey + cslots;
+  S.occ = S.ccnt + cslots;
+  S.cmask = cslots - 1;
+  uint16_t* tok = (uint16_t*)(S.occ + cslots / 32);  // token starts of one round (<= 32 per thread);
+                                                          // in the flush: the occupied slots
   const uint32_t round_stripes = 2u * (uint32_t)nthr;
-  __shared__ uint64_t nxt_item, nxt_size, nxt_base, nxt_roff;
-  __shared__ uint32_t nxt_body, page_s, used_s;
-  __shared__ uint32_t nxt_f;
-  __shared__ int32_t nxt_fd;
-  __shared__ uint32_t nocc_s, spilled_s;
+  __shared__ ItemDesc nd;  // the next item (claimed by thread 0 one item ahead)
+  __shared__ unsigned long long nxt_item;
+  __shared__ uint32_t page_s, used_s;
+  __shared__ uint32_t spilled_s;
   __shared__ uint32_t warp_tot[32];
   __shared__ unsigned long long rbase_s;
-  const uint64_t nitems = w.vars[V_NITEMS];
+  __shared__ unsigned long long nitems_s;
   ScanAcc acc{0, 0, 0};
-  // tid 0 claims the next item and loads its file fields while the block
-  // works on the current one (three dependent L2 round trips off the path)
   auto prefetch = [&]() {
     const uint64_t it = atomicAdd(&w.vars[V_NEXT], 1ull);
     nxt_item = it;
-    if (it < nitems) {
-      const ItemDesc d = w.desc[it];
-      nxt_f = d.gid;
-      nxt_fd = d.fd;
-      nxt_size = d.rlen;  // whole file: its size
-      nxt_base = (d.meta >> 31) ? ~0ull : d.roff + (d.meta & 31u);  // chunk: its start s
-      nxt_body = d.body;
-      nxt_roff = d.roff;
-    }
+    if (it < nitems_s) nd = w.desc[it];
   };
-  for (uint32_t i = tid; i < kCountSlots; i += nthr) {  // dynamic smem is not cleared between launches
+  for (uint32_t i = tid; i < cslots; i += nthr) {  // dynamic smem is not cleared between launches
     S.ckey[i] = 0;
     S.ccnt[i] = 0;
   }
+  for (uint32_t i = tid; i < cslots / 32; i += nthr) S.occ[i] = 0;
   if (tid == 0) {
+    uint64_t ni = count_items(w);
+    if (ni > w.max_items) {
+      set_err(w, -ENOSPC);
+      ni = w.max_items;
+    }
+    if (blockIdx.x == 0) w.vars[V_NITEMS] = ni;
+    nitems_s = ni;
     page_s = kNoPage;
     used_s = 0;
     prefetch();
@@ -850,102 +934,121 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __
   for (;;) {
     __syncthreads();
     lap(0);  // 0: waiting at the loop-top barrier (end of flush)
-    const uint64_t item = nxt_item;
-    if (item >= nitems) break;
-    const uint32_t f = nxt_f;
+    if (nxt_item >= nitems_s) break;
+    const ItemDesc d = nd;
+    const uint32_t f = d.gid;
     S.hf = splitmix64(f);
-    const int fd = nxt_fd;
-    const bool whole = nxt_base == ~0ull;
-    const uint64_t s = whole ? 0 : nxt_base;
-    const uint64_t e = s + (whole ? nxt_size : nxt_body);
-    const uint64_t ws = nxt_roff;
-    const uint64_t we = ws + nxt_size;  // nxt_size: the read length (rlen)
-    if (tid == 0) {
-      nocc_s = 0;
-      spilled_s = 0;
-    }
-    // file byte p lands at buf[kPre + p - s]; (dst - ws) % 16 == 0, so gread
-    // moves the span with TMA (s is a multiple of the chunk, itself of 16)
-    const uint32_t vlo = (uint32_t)(kPre - (s - ws)), vhi = vlo + (uint32_t)(we - ws);
-    // (a lane-parallel gread_lanes by warp 0 measured slower here: 23 % vs 18 % of the item time)
-    const int64_t r = gread(c, fd, ws, we - ws, S.buf + vlo);  // starts with a barrier
-    lap(1);  // 1: gread
-    if (r != (int64_t)(we - ws)) {
-      if (tid == 0) {
-        set_err(w, r < 0 ? r : -EIO);
-        prefetch();
+    const bool whole = d.meta >> 31;
+    const uint32_t nch = item_chunks(d);
+    if (tid == 0) spilled_s = 0;
+    bool bad = false;
+    for (uint32_t ci = 0; ci < nch; ++ci) {
+      const StepRange r = step_range(d, ci, chunk);
+      // file byte p lands at buf[kPre + p - s]; (dst - ws) % 16 == 0, so gread
+      // moves the span with TMA (s is a multiple of the chunk, itself of 16)
+      const uint32_t vlo = (uint32_t)(kPre - (r.s - r.ws)), vhi = vlo + (uint32_t)(r.we - r.ws);
+      // (a lane-parallel gread_lanes by warp 0 measured slower here: 23 % vs 18 % of the item time)
+      const int64_t got = gread(c, d.fd, r.ws, r.we - r.ws, S.buf + vlo);  // starts with a barrier
+      lap(1);  // 1: gread
+      if (got != (int64_t)(r.we - r.ws)) {  // the same value in every thread
+        if (tid == 0) set_err(w, got < 0 ? got : -EIO);
+        bad = true;
+        break;
       }
-      continue;
-    }
-    // pass 1: word-byte bits per 32-byte stripe; bytes outside [vlo, vhi) are non-word
-    const uint32_t nstripe = (vhi + 31) / 32;
-    for (uint32_t j = tid; j < nstripe; j += nthr)
-      S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
-    if (tid == 0) S.mask[nstripe] = 0;
-    __syncthreads();
-    lap(2);  // 2: pass 1
-    if (tid == 0) prefetch();  // next item's fields, overlapping pass 2
-    // pass 2, by rounds of 2 stripes per thread: the starts of tokens in
-    // [s, e) = buf[kPre, kPre + e - s) are compacted into `tok`, then every
-    // thread takes every nthr-th token (balanced whatever the text layout)
-    const uint32_t olo = kPre, ohi = kPre + (uint32_t)(e - s);
-    const uint32_t jlo = olo / 32, jhi = (ohi - 1) / 32;
-    for (uint32_t r0 = jlo; r0 <= jhi; r0 += round_stripes) {
-      uint32_t st[2];
-      uint32_t cnt = 0;
+      // pass 1: word-byte bits per 32-byte stripe; bytes outside [vlo, vhi) are non-word
+      const uint32_t nstripe = (vhi + 31) / 32;
+      for (uint32_t j = tid; j < nstripe; j += nthr)
+        S.mask[j] = word_bits32(S.buf + 32 * j) & bit_range((int)vlo - 32 * (int)j, (int)vhi - 32 * (int)j);
+      if (tid == 0) S.mask[nstripe] = 0;
+      __syncthreads();
+      lap(2);  // 2: pass 1
+      if (tid == 0 && ci + 1 == nch) prefetch();  // next item's descriptor, overlapping pass 2
+      // pass 2, by rounds of 2 stripes per thread: the starts of tokens in
+      // [s, e) = buf[kPre, kPre + e - s) are compacted into `tok`, then every
+      // thread takes every nthr-th token (balanced whatever the text layout)
+      const uint32_t olo = kPre, ohi = kPre + (uint32_t)(r.e - r.s);
+      const uint32_t jlo = olo / 32, jhi = (ohi - 1) / 32;
+      const uint64_t pos0 = r.s - kPre;
+      for (uint32_t r0 = jlo; r0 <= jhi; r0 += round_stripes) {
+        uint32_t st[2];
+        uint32_t cnt = 0;
 #pragma unroll
-      for (int q = 0; q < 2; ++q) {
-        const uint32_t j = r0 + 2 * (uint32_t)tid + q;
-        st[q] = 0;
-        if (j <= jhi) {
-          const uint32_t m = S.mask[j];
-          const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
-          st[q] = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
+        for (int q = 0; q < 2; ++q) {
+          const uint32_t j = r0 + 2 * (uint32_t)tid + q;
+          st[q] = 0;
+          if (j <= jhi) {
+            const uint32_t m = S.mask[j];
+            const uint32_t prev = j ? S.mask[j - 1] >> 31 : 0u;
+            st[q] = m & ~((m << 1) | prev) & bit_range((int)olo - 32 * (int)j, (int)ohi - 32 * (int)j);
+          }
+          cnt += __popc(st[q]);
         }
-        cnt += __popc(st[q]);
-      }
-      uint32_t incl = cnt;
-      for (int o = 1; o < 32; o <<= 1) {
-        const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
-        if (lane >= o) incl += t;
-      }
-      if (lane == 31) warp_tot[wid] = incl;
-      __syncthreads();
-      uint32_t off = incl - cnt, total = 0;
-      for (int q = 0; q < (nthr >> 5); ++q) {
-        const uint32_t t = warp_tot[q];
-        off += q < wid ? t : 0u;
-        total += t;
-      }
+        uint32_t incl = cnt;
+        for (int o = 1; o < 32; o <<= 1) {
+          const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+          if (lane >= o) incl += t;
+        }
+        if (lane == 31) warp_tot[wid] = incl;
+        __syncthreads();
+        uint32_t off = incl - cnt, total = 0;
+        for (int q = 0; q < (nthr >> 5); ++q) {
+          const uint32_t t = warp_tot[q];
+          off += q < wid ? t : 0u;
+          total += t;
+        }
 #pragma unroll
-      for (int q = 0; q < 2; ++q) {
-        const uint32_t jb = 32 * (r0 + 2 * (uint32_t)tid + q);
-        for (uint32_t x = st[q]; x; x &= x - 1) tok[off++] = (uint16_t)(jb + __ffs(x) - 1);
+        for (int q = 0; q < 2; ++q) {
+          const uint32_t jb = 32 * (r0 + 2 * (uint32_t)tid + q);
+          for (uint32_t x = st[q]; x; x &= x - 1) tok[off++] = (uint16_t)(jb + __ffs(x) - 1);
+        }
+        __syncthreads();
+        lap(3);  // 3: token list
+        for (uint32_t q = tid; q < total; q += nthr) {
+          const uint32_t i = tok[q], j = i >> 5, b = i & 31;
+          const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | S.mask[j];
+          const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
+          if (L <= 32)                                   // no dictionary word is longer (R12)
+            scan_token(w, S, &spilled_s, f, i, L, pos0 + i, hits, hit_cap, acc);
+        }
+        lap(4);  // 4: own tokens
+        __syncthreads();  // tok and warp_tot are reused by the next round
+        lap(5);  // 5: waiting for the block's other tokens
       }
-      __syncthreads();
-      lap(3);  // 3: token list
-      for (uint32_t q = tid; q < total; q += nthr) {
-        const uint32_t i = tok[q], j = i >> 5, b = i & 31;
-        const uint64_t win = ((uint64_t)S.mask[j + 1] << 32) | S.mask[j];
-        const uint32_t L = __ffsll(~(win >> b)) - 1;  // run of word bytes; >= 33 means too long
-        if (L <= 32)                                   // no dictionary word is longer (R12)
-          scan_token(w, S, &nocc_s, &spilled_s, f, i, L, s + i - kPre, hits, hit_cap, acc);
-      }
-      lap(4);  // 4: own tokens
-      __syncthreads();  // tok and warp_tot are reused by the next round
-      lap(5);  // 5: waiting for the block's other tokens
     }
-    // flush: a whole-file item with no spill owns its records; otherwise merge
-    const uint32_t nocc = nocc_s;
+    if (bad && tid == 0) prefetch();  // (a failed read stops before the prefetch of the last chunk)
+    // flush. The occupied slots, from the bitmap, into `tok` (free now)
+    const uint32_t nwords = cslots / 32;
+    const uint32_t wpt = (nwords + nthr - 1) / nthr, q0 = tid * wpt, q1 = min(q0 + wpt, nwords);
+    uint32_t cnt = 0;
+    for (uint32_t q = q0; q < q1; ++q) cnt += __popc(S.occ[q]);
+    uint32_t incl = cnt;
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+      if (lane >= o) incl += t;
+    }
+    if (lane == 31) warp_tot[wid] = incl;
+    __syncthreads();
+    uint32_t off = incl - cnt, nocc = 0;
+    for (int q = 0; q < (nthr >> 5); ++q) {
+      const uint32_t t = warp_tot[q];
+      off += q < wid ? t : 0u;
+      nocc += t;
+    }
+    for (uint32_t q = q0; q < q1; ++q) {
+      for (uint32_t x = S.occ[q]; x; x &= x - 1) tok[off++] = (uint16_t)(32 * q + __ffs(x) - 1);
+      S.occ[q] = 0;
+    }
+    // a whole-file item with no spill owns its records; otherwise merge
     const bool direct = whole && !spilled_s && rec;
-    if (direct && tid == 0 && nocc) rbase_s = rec_reserve(w, nocc, &page_s, &used_s);
+    if (direct && tid == 0 && nocc && !bad) rbase_s = rec_reserve(w, nocc, &page_s, &used_s);
     __syncthreads();
     if (w.prof && tid == 0) atomicAdd(&w.prof[7], 1ull);  // 7: items
     for (uint32_t q = tid; q < nocc; q += nthr) {
-      const uint32_t cs = S.olist[q];
+      const uint32_t cs = tok[q];
       const uint32_t k = S.ckey[cs] - 1, cnt = S.ccnt[cs];
       S.ckey[cs] = 0;
       S.ccnt[cs] = 0;
+      if (bad) continue;
       if (direct) {
         atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt);
         if (rbase_s != ~0ull) {
@@ -958,6 +1061,7 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __
         pair_add(w, f, k, cnt);
       }
     }
+    lap(6);  // 6: flush
   }
   if (tid == 0) rec_close(w, page_s, used_s);
   // block-level digest reduction
@@ -982,7 +1086,7 @@ __global__ void k_grep_close(const gfs_ctx* c, const __grid_constant__ GrepWork 
 }
 
 // Records of the (file, word) table (chunked files, spilled items) + their
-// word totals. A block takes 1024 consecutive slots (4 per thread, 64
+// word totals. A block takes 2048 consecutive slots (8 per thread, 128
 // contiguous bytes), reserves output space for the valid ones in its record
 // page, and empties the slots again for the next run.
 __global__ void __launch_bounds__(256) k_grep_compact(const __grid_constant__ GrepWork w, int want_rec,
@@ -996,14 +1100,15 @@ __global__ void __launch_bounds__(256) k_grep_compact(const __grid_constant__ Gr
     used_s = 0;
   }
   const uint64_t n = w.pair_mask + 1;  // a power of two >= 1024
-  for (uint64_t blk = blockIdx.x; blk * 1024 < n; blk += gridDim.x) {
-    const uint64_t i0 = blk * 1024 + (uint64_t)tid * 4;
+  constexpr int kPer = 8;                // slots per thread (128 bytes in flight per thread)
+  for (uint64_t blk = blockIdx.x; blk * 256 * kPer < n; blk += gridDim.x) {
+    const uint64_t i0 = blk * 256 * kPer + (uint64_t)tid * kPer;
     uint4* src = (uint4*)(w.pair + 2 * i0);
-    uint64_t key[4], cnt[4];
+    uint64_t key[kPer], cnt[kPer];
     uint32_t nv = 0;
 #pragma unroll
-    for (int q = 0; q < 4; ++q) {
-      const uint4 v = src[q];
+    for (int q = 0; q < kPer; ++q) {
+      const uint4 v = i0 < n ? src[q] : make_uint4(0xFFFFFFFFu, 0xFFFFFFFFu, 0u, 0u);  // (n >= 1024: whole groups)
       key[q] = ((uint64_t)v.y << 32) | v.x;
       cnt[q] = ((uint64_t)v.w << 32) | v.z;
       nv += key[q] != kPairEmpty;
@@ -1025,7 +1130,7 @@ __global__ void __launch_bounds__(256) k_grep_compact(const __grid_constant__ Gr
     __syncthreads();
     uint64_t idx = base_s + before + incl - nv;
 #pragma unroll
-    for (int q = 0; q < 4; ++q) {
+    for (int q = 0; q < kPer; ++q) {
       if (key[q] == kPairEmpty) continue;
       const uint32_t k = (uint32_t)key[q];
       atomicAdd((unsigned long long*)&totals[k], (unsigned long long)cnt[q]);
@@ -1114,12 +1219,16 @@ struct Layout {
   uint64_t off[18];
   uint64_t total;
   uint64_t max_items, tcap, pcap, max_pages;
+  uint32_t flog2;
 };
 
 Layout layout(const gfs_grep_params* p) {
   Layout L{};
   L.tcap = pow2_at_least(p->max_words * 8ull < 1024 ? 1024 : p->max_words * 8ull);
   L.pcap = pow2_at_least(p->pair_cap < 1024 ? 1024 : p->pair_cap);
+  // filter: >= 4.5 bits per word, 1 Ki .. 256 Ki bits (<= 32 KiB: it must stay in L1)
+  L.flog2 = 10;
+  while (L.flog2 < 18 && (1ull << L.flog2) < p->max_words * 9ull / 2) ++L.flog2;
   const uint64_t chunk = p->chunk ? p->chunk : 1;
   // items: one per chunk of corpus plus one partial chunk per file
   L.max_items = p->corpus_cap / chunk + p->max_files + 1;
@@ -1136,14 +1245,14 @@ Layout layout(const gfs_grep_params* p) {
       (uint64_t)p->max_files * 8,                          // 6 line_off
       (uint64_t)p->max_files * 4,                          // 7 fd
       (uint64_t)p->max_files * 8,                          // 8 size
-      ((uint64_t)p->max_files + 1) * 8,                    // 9 item_base
-      L.max_items * sizeof(ItemDesc),                      // 10 desc
-      L.pcap * 16,                                         // 11 pair
-      L.max_pages * kRecPage * 12,                         // 12 record pages
-      L.max_pages * 4,                                     // 13 page_used
-      L.max_pages * 8,                                     // 14 page_base
-      V_NVARS * 8,                                         // 15 vars
-      K_NKEEP * 8,                                         // 16 keep (persistent)
+      L.max_items * sizeof(ItemDesc),                      // 9 desc
+      L.pcap * 16,                                         // 10 pair
+      L.max_pages * kRecPage * 12,                         // 11 record pages
+      L.max_pages * 4,                                     // 12 page_used
+      L.max_pages * 8,                                     // 13 page_base
+      V_NVARS * 8,                                         // 14 vars
+      K_NKEEP * 8,                                         // 15 keep (persistent)
+      (1ull << L.flog2) / 8,                               // 16 word filter
   };
   uint64_t o = 0;
   for (int i = 0; i < 17; ++i) {
@@ -1154,10 +1263,21 @@ Layout layout(const gfs_grep_params* p) {
   return L;
 }
 
-uint32_t scan_smem(uint32_t chunk, uint32_t block) {
+uint32_t scan_smem(uint32_t chunk, uint32_t block, uint32_t cslots) {
   const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
   const uint32_t nstripe_max = (kPre + chunk + kHalo + 31) / 32;
-  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * kCountSlots * 4 + kCountSlots * 2 + 64 * block;
+  const uint32_t tok_bytes = 64 * block > 2 * cslots ? 64 * block : 2 * cslots;
+  return buf_bytes + ((nstripe_max + 1 + 3) & ~3u) * 4 + 2 * cslots * 4 + cslots / 8 + tok_bytes;
+}
+
+// Count slots per scan block: the most (<= 4096) that keep >= 768 threads of
+// the scan resident per SM (latency hiding) in 227 KiB of shared memory.
+uint32_t pick_cslots(uint32_t chunk, uint32_t block) {
+  const uint32_t blocks = (768 + block - 1) / block;
+  const uint32_t budget = 232448 / blocks - 1024 - 2048;  // per-block reserve + static shared memory
+  uint32_t cs = kMaxCountSlots;
+  while (cs > 512 && scan_smem(chunk, block, cs) > budget) cs >>= 1;
+  return cs;
 }
 
 }  // namespace
@@ -1187,18 +1307,26 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   w.file_ids = p->file_ids;
   w.fd = (int32_t*)(base + L.off[7]);
   w.size = (uint64_t*)(base + L.off[8]);
-  w.item_base = (uint64_t*)(base + L.off[9]);
-  w.desc = (ItemDesc*)(base + L.off[10]);
+  w.desc = (ItemDesc*)(base + L.off[9]);
   w.max_items = L.max_items;
   w.chunk = p->chunk;
-  w.pair = (uint64_t*)(base + L.off[11]);
+  w.cslots = pick_cslots(p->chunk, p->block);
+  {
+    // default: what the count table holds (~64 text bytes per distinct word)
+    const uint32_t wm = p->whole_max ? p->whole_max : w.cslots * 64u;
+    const uint32_t wc = wm / p->chunk;
+    w.whole_chunks = wc < kMaxWholeChunks ? wc : kMaxWholeChunks;
+  }
+  w.pair = (uint64_t*)(base + L.off[10]);
   w.pair_mask = L.pcap - 1;
-  w.rpool = (uint32_t*)(base + L.off[12]);
-  w.page_used = (uint32_t*)(base + L.off[13]);
-  w.page_base = (uint64_t*)(base + L.off[14]);
+  w.rpool = (uint32_t*)(base + L.off[11]);
+  w.page_used = (uint32_t*)(base + L.off[12]);
+  w.page_base = (uint64_t*)(base + L.off[13]);
   w.max_pages = L.max_pages;
-  w.vars = (unsigned long long*)(base + L.off[15]);
-  w.keep = (unsigned long long*)(base + L.off[16]);
+  w.vars = (unsigned long long*)(base + L.off[14]);
+  w.keep = (unsigned long long*)(base + L.off[15]);
+  w.filt = (uint32_t*)(base + L.off[16]);
+  w.filt_log2 = L.flog2;
 
   // path arguments: dictionary, list, the list's directory (relative lines)
   gfs_launch::ArgStage as(h, s);
@@ -1222,7 +1350,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
     if (d_prof) cudaMemsetAsync(d_prof, 0, 8 * sizeof(unsigned long long), s);
     w.prof = d_prof;
   }
-  const uint32_t smem = scan_smem(p->chunk, p->block);
+  const uint32_t smem = scan_smem(p->chunk, p->block, w.cslots);
   if (smem > 227 * 1024) return -EINVAL;
   cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   int dev = 0, nsm = 148;
@@ -1244,7 +1372,6 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   // gopen is collective with one leader thread: many one-warp blocks keep
   // more opens in flight (host RPCs when cold, L2 round trips when warm)
   k_grep_open<<<nsm * 16, 32, 0, s>>>(c, w, d_dir, (uint32_t)dir.size(), p->max_files);
-  k_grep_plan<<<1, 1024, 0, s>>>(w);
   k_grep_items<<<nsm * 2, 256, 0, s>>>(w);
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
   // persistent scan grid: every resident block slot once (p->grid caps it)
@@ -1266,12 +1393,12 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
     cudaMemcpyAsync(pv, w.prof, sizeof(pv), cudaMemcpyDeviceToHost, s);
     cudaStreamSynchronize(s);
     double tot = 0;
-    for (int i = 0; i < 6; ++i) tot += (double)pv[i];
+    for (int i = 0; i < 7; ++i) tot += (double)pv[i];
     tot += 1e-9;
     fprintf(stderr, "gfs_grep[scan prof, thread 0 cycles]: items=%llu loop-top=%.1f%% gread=%.1f%% pass1=%.1f%% "
-            "toklist=%.1f%% tokens=%.1f%% wait-others=%.1f%% (%.0f cycles/item)\n", pv[7], 100 * pv[0] / tot,
-            100 * pv[1] / tot, 100 * pv[2] / tot, 100 * pv[3] / tot, 100 * pv[4] / tot, 100 * pv[5] / tot,
-            tot / (double)(pv[7] ? pv[7] : 1));
+            "toklist=%.1f%% tokens=%.1f%% wait-others=%.1f%% flush=%.1f%% (%.0f cycles/item)\n", pv[7],
+            100 * pv[0] / tot, 100 * pv[1] / tot, 100 * pv[2] / tot, 100 * pv[3] / tot, 100 * pv[4] / tot,
+            100 * pv[5] / tot, 100 * pv[6] / tot, tot / (double)(pv[7] ? pv[7] : 1));
   }
   const cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) fprintf(stderr, "gfs_grep: launch failed: %s\n", cudaGetErrorString(e));

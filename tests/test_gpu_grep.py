@@ -152,3 +152,38 @@ def test_max_chunk_and_rejected_chunk(g, shmdir):
         for bad in (65536, 40):
             with pytest.raises(g.GfsError):
                 fs.grep(c["dict"], c["list"], hits=False, chunk=bad, grid=64)
+
+
+@pytest.mark.parametrize("whole_max", [1, 0, 2 * 4096, 31 * 4096])
+def test_whole_file_items_vs_oracle(g, shmdir, whole_max):
+    """Multi-chunk files of at most whole_max bytes are one work item (one block
+    scans them chunk after chunk, counting in shared memory; most chunks first);
+    larger ones are split into chunk items merged through the (file, word) table.
+    Every split (1: none whole; 0: 256 KiB; 2 and 31 chunks) is bit-exact, hits included."""
+    c = gen.c4_corpus(os.path.join(shmdir, "c4w"), seed=21, nfiles=400, total_bytes=12 << 20, nwords=3000)
+    ref = oracle.grep(c["dict"], c["list"], want_hits=True)
+    with g.GpuFS(cache_bytes=256 << 20, page_size=65536, timeout_ms=30000, daemon_threads=4,
+                 max_files=1024) as fs:
+        out = fs.grep(c["dict"], c["list"], hits=True, chunk=4096, whole_max=whole_max)
+    compare(out, ref)
+
+
+def test_whole_file_count_table_spill(g, shmdir):
+    """A whole multi-chunk file with more distinct dictionary words than the
+    per-block count table (at most 4096 slots) spills to the (file, word) table; its
+    records are then all merged there: still bit-exact."""
+    lex = gen.lexicon(6000, 7, min_len=3, max_len=12, mean=7)
+    rng = np.random.default_rng(7)
+    body = b" ".join(lex[i] for i in rng.permutation(len(lex)))
+    body = body + b"\n" + b" ".join(lex[i] for i in rng.integers(0, len(lex), 4000))
+    p0, p1 = os.path.join(shmdir, "big.txt"), os.path.join(shmdir, "small.txt")
+    open(p0, "wb").write(body)
+    open(p1, "wb").write(b" ".join(lex[:50]))
+    gen.write_dict(os.path.join(shmdir, "d.bin"), lex)
+    gen.write_list(os.path.join(shmdir, "l.txt"), [p0, p1])
+    ref = oracle.grep(os.path.join(shmdir, "d.bin"), os.path.join(shmdir, "l.txt"), want_hits=True)
+    assert len(body) <= 31 * 4096 and (ref.records[:, 0] == 0).sum() > 4096
+    with g.GpuFS(cache_bytes=64 << 20, page_size=65536, timeout_ms=30000, daemon_threads=2) as fs:
+        out = fs.grep(os.path.join(shmdir, "d.bin"), os.path.join(shmdir, "l.txt"), hits=True, chunk=4096,
+                      whole_max=31 * 4096, grid=4)
+    compare(out, ref)
