@@ -183,9 +183,11 @@ int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint64_t file
 /* Cache-hit read benchmark (K4 shape): block b issues
  * calls_per_block greads of `chunk` bytes into dynamic shared memory at file
  * offsets d_off[b*calls_per_block + i] (chunk-aligned), checksumming each
- * chunk from shared memory into *d_sum. raw != 0 runs the baseline: the same
- * copies straight from d_raw (the file's bytes already in device memory),
- * without GPUfs (h may be NULL then). */
+ * chunk from shared memory into *d_sum. raw: 0 = gread; 1 = the baseline: the
+ * same copies straight from d_raw (the file's bytes already in device memory),
+ * without GPUfs (h may be NULL then); 2 = gread_hint, each call naming the
+ * block's next offset (split-phase lookup: the next page is looked up and
+ * referenced while the current copy is in flight). */
 int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
                      uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
                      int64_t* d_err, uint32_t grid, uint32_t block);

@@ -225,7 +225,9 @@ __device__ __forceinline__ void backoff(uint32_t& ns) {
 }
 
 __device__ __forceinline__ void ctr(const gfs_ctx* c, int i, unsigned long long v = 1) {
+#ifndef GFS_NO_COUNTERS  // (diagnostic builds only: measures what the statistics cost)
   red_add64(&c->ctr[(size_t)i * GFS_CTR_SHARDS + (smid() & (GFS_CTR_SHARDS - 1))], v);
+#endif
 }
 
 __device__ __forceinline__ uint32_t stamp_now() { return (uint32_t)(now_ns() >> 10); }
@@ -296,6 +298,14 @@ struct Scratch {
   uint32_t ra_n;
   uint32_t ra_f[16];
   uint64_t ra_v[16];
+  // next-call hint (gread_hint): a page of the block's next gread, looked up
+  // and referenced while this call's copy was in flight; valid for hint_grid
+  // / hint_blk while hint_f >= 0, consumed or released by the next gread/gclose
+  uint64_t hint_grid;
+  uint32_t hint_blk;
+  int32_t hint_fd;
+  int32_t hint_f;
+  uint64_t hint_page;
 };
 constexpr uint32_t kRA = 16;  // read-ahead fills a block tracks
 
@@ -2123,6 +2133,12 @@ __device__ inline int gclose_t(const gfs_ctx* c, int fd) {
   }
   if (G::tid() == 0) {
     if (sc.cached_fd == fd) sc.cached_fd = -1;
+    if constexpr (G::kBlock) {  // an unconsumed gread hint on this file
+      if (sc.hint_grid == detail::grid_id() && sc.hint_blk == G::key() && sc.hint_f >= 0 && sc.hint_fd == fd) {
+        detail::r64_add_rlx(&c->f_state[sc.hint_f], detail::kRefDec);
+        sc.hint_f = -1;
+      }
+    }
     sc.ret = detail::close_leader(c, fd);
   }
   G::sync();
@@ -2215,7 +2231,8 @@ __device__ __noinline__ int64_t gread_batches(const gfs_ctx* c, int64_t n, uint6
 
 // gread: pread semantics; returns min(len, S-off) bytes, 0 at/after EOF.
 template <class G>
-__device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
+__device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst,
+                                  uint64_t next_off = ~0ull) {
   using namespace detail;
   Scratch& sc = G::sc();
   const int tid = G::tid(), nthr = G::nthr();
@@ -2245,12 +2262,21 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
     __syncwarp(nthr >= 32 ? 0xFFFFFFFFu : ((1u << nthr) - 1u));
     const int64_t n0 = sc.ret;
     uint32_t quick = 0;
+    // the previous call's hint: this call's first page, already referenced
+    int hinted = -1;
+    if constexpr (G::kBlock) {
+      if (tid == 0 && sc.hint_grid == grid_id() && sc.hint_blk == G::key() && sc.hint_f >= 0) {
+        if (n0 > 0 && sc.hint_fd == fd && sc.hint_page == (off >> shift)) hinted = sc.hint_f;
+        else r64_add_rlx(&c->f_state[sc.hint_f], kRefDec);  // not this call's: drop it
+        sc.hint_f = -1;
+      }
+    }
     if (n0 > 0) {
       const uint64_t q0 = off >> shift, q1 = (off + (uint64_t)n0 - 1) >> shift;
       const uint32_t cnt = (uint32_t)((q1 - q0 + 1) < B ? (q1 - q0 + 1) : B);
       if (tid < (int)cnt) {
         const FileSnap fs0 = sc.fs;
-        int f = fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
+        int f = hinted >= 0 ? hinted : fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
         if (f < 0) {
           const Lk r = lookup_try(c, fs0, q0 + tid);
           sc.frame[tid] = r.frame;
@@ -2285,6 +2311,16 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
   if (sc.quick) {
     const uint32_t ph = sc.mbar_phase;
     copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + (off & (P - 1)), (uint32_t)n, tid);
+    if constexpr (G::kBlock) {
+      // hint: look up and reference the next call's first page while the copy flies
+      if (next_off != ~0ull && tid == 0 && fast && next_off < sc.fs.size) {
+        sc.hint_grid = grid_id();
+        sc.hint_blk = G::key();
+        sc.hint_fd = fd;
+        sc.hint_page = next_off >> shift;
+        sc.hint_f = lookup_fast(c, sc.fs, sc.hint_page, sc.lc_ok ? sc.leaf : nullptr);
+      }
+    }
     mbar_wait(&sc.mbar, ph);
     G::sync();
     if (tid == 0) {
@@ -2310,6 +2346,16 @@ __device__ inline int gclose(const gfs_ctx* c, int fd) { return gclose_t<detail:
 __device__ inline int64_t gfstat_size(const gfs_ctx* c, int fd) { return gfstat_size_t<detail::BlockGroup>(c, fd); }
 __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst) {
   return gread_t<detail::BlockGroup>(c, fd, off, len, dst);
+}
+// gread with the offset of the block's NEXT gread on the same file (a split-
+// phase lookup, NEXT-2): while this call's one-page copy into
+// shared memory is in flight, warp 0 looks up and references the page holding
+// next_off, so the next call starts its copy without a lookup. The reference
+// is consumed by the next gread (or dropped by it if the offset differs) or by
+// gclose: a block that passes a hint must call gread or gclose again.
+__device__ inline int64_t gread_hint(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst,
+                                     uint64_t next_off) {
+  return gread_t<detail::BlockGroup>(c, fd, off, len, dst, next_off);
 }
 
 // Warp-collective calls (the paper's design point): every lane of

@@ -163,9 +163,10 @@ class GpuFS:
 
     # cache-hit reads into shared memory (K4) ---------------------------------
     def randread(self, path, chunk, offs, grid, block=256, raw=None, stream=None, sync=True, out=None, warp=False,
-                 depth=0):
+                 depth=0, hint=False):
         """K4 reads into shared memory; warp: the warp-collective calls; depth > 0: the split-phase
-        lane-parallel calls, `depth` of them in flight per block (gfs_run_randread_async)."""
+        lane-parallel calls, `depth` of them in flight per block (gfs_run_randread_async); hint: every
+        call names the block's next offset (gread_hint: the next lookup overlaps this copy)."""
         torch = _torch()
         dev = f"cuda:{self.device}"
         if isinstance(offs, torch.Tensor):
@@ -188,7 +189,7 @@ class GpuFS:
             v = out.cpu().numpy()
             return int(v[0].astype(np.uint64)), int(v[1])
         fn = gfs_run_randread_warp if warp else gfs_run_randread
-        fn(self.h, sp, path, 1 if raw is not None else 0,
+        fn(self.h, sp, path, 1 if raw is not None else (2 if hint and not warp else 0),
                          raw.data_ptr() if raw is not None else None, chunk, calls, d_off.data_ptr(),
                          out.data_ptr(), out.data_ptr() + 8, grid, block)
         if not sync:

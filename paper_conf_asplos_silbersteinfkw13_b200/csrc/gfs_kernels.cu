@@ -223,6 +223,8 @@ __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const cha
   extern __shared__ __align__(16) uint8_t smem[];
   const int tid = threadIdx.x, nthr = blockDim.x;
   int fd = 0;
+  const bool hint = raw == 2;
+  raw = raw == 1;
   if (!raw) {
     fd = gopen(c, path, GFS_O_RDONLY);
     if (fd < 0) {
@@ -255,7 +257,8 @@ __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const cha
       __syncthreads();
       r = chunk;
     } else {
-      r = gread(c, fd, o, chunk, smem);
+      r = hint ? gread_hint(c, fd, o, chunk, smem, i + 1 < calls ? my[i + 1] : ~0ull)
+                   : gread(c, fd, o, chunk, smem);
       if (r < 0) {
         if (tid == 0) note_err(err, r);
         break;
@@ -560,16 +563,16 @@ GFS_API int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint6
 GFS_API int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, const uint8_t* d_raw,
                              uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
                              int64_t* d_err, uint32_t grid, uint32_t block) {
-  if ((!raw && !h) || (raw && !d_raw) || grid == 0 || block == 0 || chunk == 0 || (chunk & 15) ||
-      chunk > 200 * 1024)
+  if (raw < 0 || raw > 2 || (raw != 1 && !h) || (raw == 1 && !d_raw) || grid == 0 || block == 0 || chunk == 0 ||
+      (chunk & 15) || chunk > 200 * 1024)
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
-  gfs_launch::ArgStage as(raw ? nullptr : h, s);
-  if (!raw)
+  gfs_launch::ArgStage as(raw == 1 ? nullptr : h, s);
+  if (raw != 1)
     if (const int e = as.stage(&path, 1)) return e;
-  const char* dp = raw ? nullptr : as.str(0);
+  const char* dp = raw == 1 ? nullptr : as.str(0);
   if (chunk > 48 * 1024) cudaFuncSetAttribute(k_randread, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
-  k_randread<<<grid, block, chunk, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
+  k_randread<<<grid, block, chunk, s>>>(raw == 1 ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
                                         d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }

@@ -279,3 +279,30 @@ def test_zero_copy_registered_file(g, shmdir, P):
     with pytest.raises(g.GfsError):
         with _fs(g, cache_bytes=4 * P, page_size=P) as fs2:
             fs2.register_file(os.path.join(shmdir, "missing.bin"))
+
+
+def test_randread_hint_checksum_and_no_leaked_references(g, shmdir):
+    """gread_hint (each call names the block's next offset; its page is looked up
+    and referenced while the current copy flies): same bytes as plain gread, warm
+    and in a cache too small to hold the file (hints then miss or get evicted
+    before use), and no reference outlives the kernel: a sweep that needs every
+    frame of the tiny cache afterwards still completes."""
+    P = 1 << 16
+    size = 64 * P
+    chunk = 16384
+    path = gen.splitmix_file(os.path.join(shmdir, "k4h.bin"), size, seed=33)
+    other = gen.splitmix_file(os.path.join(shmdir, "k4h2.bin"), size, seed=34)
+    grid, calls = 16, 40
+    rng = np.random.default_rng(3)
+    offs = (rng.integers(0, size // chunk, size=grid * calls) * chunk).astype(np.uint64)
+    offs[5] = offs[4]  # a hint for the page the block already holds
+    expect = sum(oracle.checksum(path, int(o), chunk) for o in offs) % (1 << 64)
+    with _fs(g, cache_bytes=128 * P, page_size=P) as fs:  # the file fits: warm hits
+        assert fs.randread(path, chunk, offs, grid) == (expect, 0)
+        assert fs.randread(path, chunk, offs, grid, hint=True) == (expect, 0)
+        assert fs.randread(path, chunk, offs, grid, block=128, hint=True) == (expect, 0)
+    with _fs(g, cache_bytes=24 * P, page_size=P) as fs:  # 24 frames for 64 pages: churn
+        for _ in range(2):
+            assert fs.randread(path, chunk, offs, grid, hint=True) == (expect, 0)
+        s, err = fs.seqread(other, size, P, grid=24)
+        assert err == 0 and s == oracle.checksum(other, 0, size)
