@@ -2230,7 +2230,7 @@ __device__ __noinline__ int64_t gread_batches(const gfs_ctx* c, int64_t n, uint6
 }
 
 // gread: pread semantics; returns min(len, S-off) bytes, 0 at/after EOF.
-template <class G>
+template <class G, bool kHint = false>
 __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst,
                                   uint64_t next_off = ~0ull) {
   using namespace detail;
@@ -2264,7 +2264,7 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
     uint32_t quick = 0;
     // the previous call's hint: this call's first page, already referenced
     int hinted = -1;
-    if constexpr (G::kBlock) {
+    if constexpr (G::kBlock && kHint) {
       if (tid == 0 && sc.hint_grid == grid_id() && sc.hint_blk == G::key() && sc.hint_f >= 0) {
         if (n0 > 0 && sc.hint_fd == fd && sc.hint_page == (off >> shift)) hinted = sc.hint_f;
         else r64_add_rlx(&c->f_state[sc.hint_f], kRefDec);  // not this call's: drop it
@@ -2311,7 +2311,7 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
   if (sc.quick) {
     const uint32_t ph = sc.mbar_phase;
     copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + (off & (P - 1)), (uint32_t)n, tid);
-    if constexpr (G::kBlock) {
+    if constexpr (G::kBlock && kHint) {
       // hint: look up and reference the next call's first page while the copy flies
       if (next_off != ~0ull && tid == 0 && fast && next_off < sc.fs.size) {
         sc.hint_grid = grid_id();
@@ -2351,11 +2351,13 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
 // phase lookup, NEXT-2): while this call's one-page copy into
 // shared memory is in flight, warp 0 looks up and references the page holding
 // next_off, so the next call starts its copy without a lookup. The reference
-// is consumed by the next gread (or dropped by it if the offset differs) or by
-// gclose: a block that passes a hint must call gread or gclose again.
+// is consumed by the next gread_hint (or dropped by it if the offset differs;
+// next_off = ~0: no further hint) or by gclose of the file. Plain gread does
+// not look at hints (it pays nothing for them), so a block that passed a hint
+// calls gread_hint or gclose next.
 __device__ inline int64_t gread_hint(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst,
                                      uint64_t next_off) {
-  return gread_t<detail::BlockGroup>(c, fd, off, len, dst, next_off);
+  return gread_t<detail::BlockGroup, true>(c, fd, off, len, dst, next_off);
 }
 
 // Warp-collective calls (the paper's design point): every lane of

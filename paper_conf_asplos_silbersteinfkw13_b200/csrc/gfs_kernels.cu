@@ -218,12 +218,12 @@ __global__ void __launch_bounds__(256, 4) k_seqread(const gfs_ctx* c, const char
   gclose(c, fd);
 }
 
+template <bool kHint>
 __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const char* path, int raw, const uint8_t* rawp, uint32_t chunk,
                            uint32_t calls, const uint64_t* offs, uint64_t* sum, int64_t* err) {
   extern __shared__ __align__(16) uint8_t smem[];
   const int tid = threadIdx.x, nthr = blockDim.x;
   int fd = 0;
-  const bool hint = raw == 2;
   raw = raw == 1;
   if (!raw) {
     fd = gopen(c, path, GFS_O_RDONLY);
@@ -257,8 +257,8 @@ __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const cha
       __syncthreads();
       r = chunk;
     } else {
-      r = hint ? gread_hint(c, fd, o, chunk, smem, i + 1 < calls ? my[i + 1] : ~0ull)
-                   : gread(c, fd, o, chunk, smem);
+      if constexpr (kHint) r = gread_hint(c, fd, o, chunk, smem, i + 1 < calls ? my[i + 1] : ~0ull);
+      else r = gread(c, fd, o, chunk, smem);
       if (r < 0) {
         if (tid == 0) note_err(err, r);
         break;
@@ -571,9 +571,10 @@ GFS_API int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int 
   if (raw != 1)
     if (const int e = as.stage(&path, 1)) return e;
   const char* dp = raw == 1 ? nullptr : as.str(0);
-  if (chunk > 48 * 1024) cudaFuncSetAttribute(k_randread, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
-  k_randread<<<grid, block, chunk, s>>>(raw == 1 ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
-                                        d_off, d_sum, d_err);
+  auto kern = raw == 2 ? k_randread<true> : k_randread<false>;
+  if (chunk > 48 * 1024) cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
+  kern<<<grid, block, chunk, s>>>(raw == 1 ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
+                                  d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
 
