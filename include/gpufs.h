@@ -192,6 +192,14 @@ int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int raw, con
                      uint32_t chunk, uint32_t calls_per_block, const uint64_t* d_off, uint64_t* d_sum,
                      int64_t* d_err, uint32_t grid, uint32_t block);
 
+/* Host->device link probe (the miss path's roofline): best of `reps` over
+ * nbytes (>= 1 MiB, multiple of 16) of mapped pinned host memory, moved (a) by
+ * the copy engine (cudaMemcpyAsync) into *ce_gbps and (b) by SMs pulling
+ * 16-byte words (__ldcv, as gread pulls staging slots) into *sm_gbps, in
+ * GB/s (1e9 B/s). Allocates and frees its own buffers; synchronises `stream`.
+ * -EINVAL on bad arguments, -ENOMEM if the buffers cannot be allocated. */
+int gfs_probe_h2d(void* stream, uint64_t nbytes, uint32_t reps, double* ce_gbps, double* sm_gbps);
+
 /* The same benchmark with the warp-collective API (gread_warp):
  * block/32 warps per block, each with its own `chunk` bytes of shared memory,
  * warp w of block b issuing calls w, w + block/32, ... of block b's

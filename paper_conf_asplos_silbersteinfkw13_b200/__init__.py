@@ -95,6 +95,7 @@ def lib():
             "gfs_run_gread": ([P, P, CS, I, U32, P, P, P, P, P, U32, U32, U32], I),
             "gfs_run_seqread": ([P, P, CS, U64, U64, U64, I, P, P, P, U32, U32], I),
             "gfs_run_randread": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
+            "gfs_probe_h2d": ([P, U64, U32, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_double)], I),
             "gfs_run_randread_warp": ([P, P, CS, I, P, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_randread_async": ([P, P, CS, I, P, U32, U32, U32, P, P, P, U32, U32], I),
             "gfs_run_gwrite": ([P, P, CS, U32, P, P, P, P, P, U32, U32, I], I),
@@ -201,6 +202,13 @@ def gfs_run_gread(h, stream, path, mode, ncalls, d_off, d_len, d_dstoff, d_dst, 
 def gfs_run_seqread(h, stream, path, file_off, total, chunk, use_mmap, d_scratch, d_sum, d_err, grid, block):
     return _ck(lib().gfs_run_seqread(h, stream, _b(path), file_off, total, chunk, use_mmap, d_scratch, d_sum,
                                      d_err, grid, block), "gfs_run_seqread")
+
+
+def gfs_probe_h2d(stream, nbytes=256 << 20, reps=10):
+    """(copy-engine GB/s, SM-pull GB/s) of the host->device link (include/gpufs.h)."""
+    ce, sm = ctypes.c_double(0), ctypes.c_double(0)
+    _ck(lib().gfs_probe_h2d(stream, nbytes, reps, ctypes.byref(ce), ctypes.byref(sm)), "gfs_probe_h2d")
+    return ce.value, sm.value
 
 
 def gfs_run_randread(h, stream, path, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err, grid, block):

@@ -9,6 +9,8 @@
 //   k_gwrite_calls    gwrite harness (O_GWRONCE)
 //   k_fileop          gfsync / gftruncate / gfstat / gopen+gclose
 #include <cuda_runtime.h>
+
+#include <algorithm>
 #include <errno.h>
 #include <stdint.h>
 #include <string.h>
@@ -675,4 +677,55 @@ GFS_API int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int fl
   }
   k_fileop<<<1, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, op, arg, d_ret);
   return launch_err(cudaGetLastError());
+}
+
+// ------------------------------------------------------------------ link probe
+// The host->device link as the miss path uses it: SMs pulling 16-byte words
+// from mapped pinned host memory (__ldcv, like the staging pull), next to the
+// copy engine's cudaMemcpyAsync. The roofline of the miss path is the faster.
+__global__ void __launch_bounds__(256) k_link_pull(const int4* src, int4* dst, uint64_t n16) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n16; i += stride) dst[i] = __ldcv(src + i);
+}
+
+GFS_API int gfs_probe_h2d(void* stream, uint64_t nbytes, uint32_t reps, double* ce_gbps, double* sm_gbps) {
+  if (!ce_gbps || !sm_gbps || nbytes < (1u << 20) || (nbytes & 15) || reps == 0) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  uint8_t *h = nullptr, *hd = nullptr, *d = nullptr;
+  if (cudaHostAlloc((void**)&h, nbytes, cudaHostAllocMapped | cudaHostAllocPortable) != cudaSuccess) return -ENOMEM;
+  memset(h, 1, nbytes);  // first touch: the pages exist before the timed copies
+  if (cudaHostGetDevicePointer((void**)&hd, h, 0) != cudaSuccess || cudaMalloc((void**)&d, nbytes) != cudaSuccess) {
+    cudaFreeHost(h);
+    return -ENOMEM;
+  }
+  int dev = 0, nsm = 148;
+  cudaGetDevice(&dev);
+  cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
+  cudaEvent_t e0, e1;
+  cudaEventCreate(&e0);
+  cudaEventCreate(&e1);
+  double best_ce = 0, best_sm = 0;
+  for (uint32_t r = 0; r < reps; ++r) {
+    float ms = 0;
+    cudaEventRecord(e0, s);
+    cudaMemcpyAsync(d, h, nbytes, cudaMemcpyHostToDevice, s);
+    cudaEventRecord(e1, s);
+    cudaEventSynchronize(e1);
+    cudaEventElapsedTime(&ms, e0, e1);
+    if (ms > 0) best_ce = std::max(best_ce, nbytes / (ms * 1e6));
+    cudaEventRecord(e0, s);
+    k_link_pull<<<nsm * 8, 256, 0, s>>>((const int4*)hd, (int4*)d, nbytes / 16);
+    cudaEventRecord(e1, s);
+    cudaEventSynchronize(e1);
+    cudaEventElapsedTime(&ms, e0, e1);
+    if (ms > 0) best_sm = std::max(best_sm, nbytes / (ms * 1e6));
+  }
+  const cudaError_t e = cudaGetLastError();
+  cudaEventDestroy(e0);
+  cudaEventDestroy(e1);
+  cudaFree(d);
+  cudaFreeHost(h);
+  *ce_gbps = best_ce;
+  *sm_gbps = best_sm;
+  return e == cudaSuccess ? 0 : -EIO;
 }
