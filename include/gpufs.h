@@ -289,7 +289,10 @@ typedef struct gfs_grep_params {
                            slots being what shared memory allows at >= 768 threads per SM:
                            4096 at block 256 / chunk 16 KiB, 1024 at block 128; <= chunk: never). Larger
                            files are split into chunk items merged through the (file, word) table */
-  uint32_t pad0;
+  uint32_t scan;        /* 0: block scan (one block per item, items staged in shared memory by
+                           gread/TMA); 1: warp scan (one warp per item, no block barrier, the
+                           text read in place through gmmap_warp; needs chunk a multiple of 1024
+                           and <= 65536, whole_max <= 65536, max_words < 65535) */
 } gfs_grep_params;
 
 /* Device scratch bytes gfs_grep needs for these parameters. */

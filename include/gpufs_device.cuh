@@ -14,6 +14,11 @@
 //   int64_t gfstat_size(const gfs_ctx*, int fd);
 //   int     gftruncate(const gfs_ctx*, int fd, uint64_t size);
 //
+// Warp-collective variants (the paper's warp granularity):
+// gopen_warp, gclose_warp, gfstat_size_warp, gread_warp, gmmap_warp,
+// gmunmap_warp (same arguments and semantics, one warp instead of the block),
+// and the vectored gread_lanes (one request per lane).
+//
 // Calling convention (§4): every thread of the threadblock calls
 // the same function with the same arguments at the same point; each call is an
 // implicit barrier and every thread receives the same return value. Negative
@@ -2729,35 +2734,37 @@ __device__ inline int gfsync(const gfs_ctx* c, int fd) {
 // gmmap: map a prefix of at most one cache page;
 // returns a pointer straight into the frame, NULL at/after EOF
 // or on error. *mapped_len = min(len, P - off%P, S - off). MAP_FIXED (addr) is
-// ignored; prot is not enforced.
-__device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int prot, int flags, int fd, uint64_t off,
-                              uint64_t* mapped_len) {
+// ignored; prot is not enforced. Group-collective
+// (G = block or warp); *err_out (optional) gets 0 or the -errno of a NULL.
+template <class G>
+__device__ inline void* gmmap_t(const gfs_ctx* c, void* addr, uint64_t len, int prot, int flags, int fd, uint64_t off,
+                                uint64_t* mapped_len, int* err_out = nullptr) {
   using namespace detail;
   (void)addr;
   (void)flags;
-  Scratch& sc = scratch();
-  const int tid = block_tid();
+  Scratch& sc = G::sc();
+  const int tid = G::tid();
   const bool wmap = (prot & (int)GFS_PROT_WRITE) != 0;
-  __syncthreads();
+  G::sync();
   if (tid == 0) {
     FileSnap s;
     sc.ptr = nullptr;
     sc.aux = 0;
     sc.ret = 0;
-    if (!snap_fd_cached(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE) || (wmap && !(s.oflags & GFS_O_RDWR))) {
+    if (!snap_fd_cached<G>(c, sc, fd, &s) || (s.oflags & GFS_O_GWRONCE) || (wmap && !(s.oflags & GFS_O_RDWR))) {
       sc.aux = -EBADF;  // a writable mapping needs an O_RDWR file
     } else if (off < s.size && len > 0) {
       sc.fs = s;
-      sc.lc_ok = (sc.cached_fd == fd && sc.cached_blk == block_linear() && sc.cached_grid == grid_id()) ? 1u : 0u;
+      sc.lc_ok = (sc.cached_fd == fd && sc.cached_blk == G::key() && sc.cached_grid == grid_id()) ? 1u : 0u;
       sc.ret = 1;
     }
   }
-  __syncthreads();
+  G::sync();
   if (sc.ret == 1) {
     const FileSnap fs = sc.fs;
-    int err = acquire_batch(c, sc, fs, off >> c->page_shift, 1, false);
+    int err = acquire_batch<G>(c, sc, fs, off >> c->page_shift, 1, false);
     if (!err && wmap) {  // writes through the pointer are untracked: keep the pristine copy, mark the range dirty
-      err = ensure_pristine(c, sc, fs.fdx, 1);
+      err = ensure_pristine<G>(c, sc, fs.fdx, 1);
       if (tid == 0) {
         if (err) {
           frame_release(c, (uint32_t)sc.frame[0]);
@@ -2784,30 +2791,54 @@ __device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int pr
         sc.aux = (int64_t)m;
       }
     }
-    __syncthreads();
+    G::sync();
   }
   if (mapped_len) *mapped_len = sc.aux > 0 ? (uint64_t)sc.aux : 0;
-  return sc.ptr;
+  if (err_out) *err_out = sc.aux < 0 ? (int)sc.aux : 0;
+  void* const r = sc.ptr;
+  if constexpr (!G::kBlock) __syncwarp();  // sc is reused by the warp's next call
+  return r;
 }
 
 // gmunmap: release the page reference; the frame is found from the pointer
 // (i-th pframe <-> i-th page).
-__device__ inline int gmunmap(const gfs_ctx* c, void* addr, uint64_t len) {
+template <class G>
+__device__ inline int gmunmap_t(const gfs_ctx* c, void* addr, uint64_t len) {
   using namespace detail;
   (void)len;
-  Scratch& sc = scratch();
-  __syncthreads();
-  if (block_tid() == 0) {
-    const uint8_t* p = (const uint8_t*)addr;
-    if (p < c->pool || p >= c->pool + ((size_t)c->nframes << c->page_shift)) {
-      sc.ret = -EINVAL;
-    } else {
-      frame_release(c, (uint32_t)((size_t)(p - c->pool) >> c->page_shift));
-      sc.ret = 0;
+  const uint8_t* p = (const uint8_t*)addr;
+  const bool ok = p >= c->pool && p < c->pool + ((size_t)c->nframes << c->page_shift);
+  if constexpr (G::kBlock) {
+    Scratch& sc = G::sc();
+    __syncthreads();
+    if (block_tid() == 0) {
+      if (ok) frame_release(c, (uint32_t)((size_t)(p - c->pool) >> c->page_shift));
+      sc.ret = ok ? 0 : -EINVAL;
     }
+    __syncthreads();
+    return (int)sc.ret;
+  } else {  // the pointer is the same in every lane: no scratch round trip
+    __syncwarp();
+    if (ok && G::tid() == 0) frame_release(c, (uint32_t)((size_t)(p - c->pool) >> c->page_shift));
+    return ok ? 0 : -EINVAL;
   }
-  __syncthreads();
-  return (int)sc.ret;
+}
+
+__device__ inline void* gmmap(const gfs_ctx* c, void* addr, uint64_t len, int prot, int flags, int fd, uint64_t off,
+                              uint64_t* mapped_len) {
+  return gmmap_t<detail::BlockGroup>(c, addr, len, prot, flags, fd, off, mapped_len);
+}
+__device__ inline int gmunmap(const gfs_ctx* c, void* addr, uint64_t len) {
+  return gmunmap_t<detail::BlockGroup>(c, addr, len);
+}
+// Warp-collective gmmap / gmunmap (the paper's warp granularity):
+// same semantics; a warp holds its mappings independently of the other warps.
+__device__ inline void* gmmap_warp(const gfs_ctx* c, void* addr, uint64_t len, int prot, int flags, int fd,
+                                   uint64_t off, uint64_t* mapped_len) {
+  return gmmap_t<detail::WarpGroup>(c, addr, len, prot, flags, fd, off, mapped_len);
+}
+__device__ inline int gmunmap_warp(const gfs_ctx* c, void* addr, uint64_t len) {
+  return gmunmap_t<detail::WarpGroup>(c, addr, len);
 }
 
 // gmsync: write back the dirty page mapped at `addr` now (Tab.1), for a

@@ -53,7 +53,7 @@ class gfs_grep_params(ctypes.Structure):
                 ("pair_cap", ctypes.c_uint64), ("hit_cap", ctypes.c_uint64), ("chunk", ctypes.c_uint32),
                 ("grid", ctypes.c_uint32), ("block", ctypes.c_uint32), ("keep_open", ctypes.c_uint32),
                 ("corpus_cap", ctypes.c_uint64), ("file_ids", ctypes.c_void_p), ("rec_cap", ctypes.c_uint64),
-                ("whole_max", ctypes.c_uint32), ("pad0", ctypes.c_uint32)]
+                ("whole_max", ctypes.c_uint32), ("scan", ctypes.c_uint32)]
 
 
 class gfs_export_desc(ctypes.Structure):

@@ -243,13 +243,13 @@ class GpuFS:
     # grep -w ------------------------------------------------------------------
     def grep_state(self, dict_path, list_path, hits=False, chunk=16384, grid=None, block=128, keep_open=False,
                    pair_cap=1 << 23, hit_cap=None, corpus_cap=1 << 34, rec_cap=1 << 22, file_ids=None,
-                   whole_max=0):
+                   whole_max=0, scan=0):
         """Device buffers of one grep configuration (allocated once, reused by grep(state=...)).
         Capacities come from file metadata (stat), never from file contents. file_ids: optional
         per-list-line ids reported instead of the line index (e.g. a shard's global file indices).
         whole_max: files of more than one chunk and at most this many bytes are scanned whole by
         one block (0: what the block's count table holds, 64 bytes per slot; <= chunk: every
-        multi-chunk file is split)."""
+        multi-chunk file is split). scan: 0 block scan, 1 warp scan (include/gpufs.h)."""
         import os
         torch = _torch()
         from . import gfs_grep_params, gfs_grep_work_bytes
@@ -259,7 +259,7 @@ class GpuFS:
         p = gfs_grep_params(max_files=max(1, lbytes // 2 + 1), max_words=nwords, list_cap=max(lbytes, 1),
                             pair_cap=pair_cap, hit_cap=0, chunk=chunk, grid=grid or 1 << 20, block=block,
                             keep_open=1 if keep_open else 0, corpus_cap=corpus_cap, rec_cap=rec_cap,
-                            whole_max=whole_max)
+                            whole_max=whole_max, scan=scan)
         d_ids = None
         if file_ids is not None:
             d_ids = torch.as_tensor(np.ascontiguousarray(np.asarray(file_ids, dtype=np.uint32)).view(np.int32),
@@ -276,7 +276,7 @@ class GpuFS:
 
     def grep(self, dict_path, list_path, hits=False, chunk=16384, grid=None, block=128, keep_open=False,
              pair_cap=1 << 23, hit_cap=None, stream=None, sync=True, state=None, corpus_cap=1 << 34,
-             rec_cap=1 << 22, file_ids=None, whole_max=0):
+             rec_cap=1 << 22, file_ids=None, whole_max=0, scan=0):
         """grep -w. Returns a dict with records (n,3) sorted by (file, word),
         totals, digest (sum, xor, nhits), hits (n,3) sorted by (file, offset, word) if requested.
         With sync=False, only enqueues and returns the state (read it after synchronising).
@@ -286,7 +286,7 @@ class GpuFS:
         from . import GREP_SUMMARY, gfs_grep
         if state is None:
             state = self.grep_state(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap, hit_cap,
-                                    corpus_cap, rec_cap, file_ids, whole_max)
+                                    corpus_cap, rec_cap, file_ids, whole_max, scan)
         p = state["p"]
         s, sp = self._stream(stream)
         gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
@@ -299,7 +299,7 @@ class GpuFS:
         if summ["err"] == -28 and pair_cap < (1 << 30):  # -ENOSPC: a table was too small
             return self.grep(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap * 4, hit_cap,
                              stream, sync, None, corpus_cap * 4, max(rec_cap, summ["nrecords"]) * 2, file_ids,
-                             whole_max)
+                             whole_max, scan)
         out = {"summary": summ}
         nrec = min(summ["nrecords"], state["rec_cap"])
         r = state["rec"][:3 * nrec].view(nrec, 3).cpu().numpy().astype(np.uint64)

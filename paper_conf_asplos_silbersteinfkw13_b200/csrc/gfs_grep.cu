@@ -125,7 +125,8 @@ enum { V_NFILES = 0, V_NWORDS, V_NITEMS, V_NEXT, V_ERR, V_BYTES, V_NREC, V_NHITS
        V_CUR_ONE,                          // one-chunk files: placement cursor = their count
        V_WHOLE_HIST,                       // [n]: multi-chunk whole files of n chunks
        V_WHOLE_CUR = V_WHOLE_HIST + kMaxWholeChunks + 1,  // [n]: their placement cursors
-       V_NVARS = V_WHOLE_CUR + kMaxWholeChunks + 1 };
+       V_NDIRECT = V_WHOLE_CUR + kMaxWholeChunks + 1,  // records the warp scan wrote straight into d_rec
+       V_NVARS };
 enum { K_MAGIC = 0, K_PAIRS, K_DICT_FD, K_LIST_FD, K_NKEEP };
 
 __device__ __forceinline__ bool is_word(uint32_t ch) {
@@ -1077,6 +1078,376 @@ __global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __
   }
 }
 
+// --------------------------------------------------------------- warp scan
+// The warp-granularity scan (gfs_grep_params.scan = 1; the paper's API
+// granularity is the warp): every warp pulls its own items and
+// works through them with no block barrier. A warp maps the item's pages with
+// gmmap_warp (zero copy: the text is read straight out of the cache frames,
+// P:L426-441) and walks the item in 1 KiB steps, 32 bytes per lane:
+//   - the next step's 32 bytes per lane are loaded while this step is scanned;
+//   - each lane classifies its 32 bytes in registers (word_bits4), token
+//     starts come from the masks and the previous lane's last bit (shuffle);
+//   - the step (+ 64 lookahead bytes) is staged in the warp's shared buffer,
+//     the token starts compacted into a list (warp prefix sum), and lanes take
+//     every 32nd token: hash, L1 filter, one 32-byte bucket of the table, and
+//     an exact 32-byte compare on a fingerprint match (as k_grep_scan);
+//   - hits count in the warp's own shared table of packed (word + 1) << 16 |
+//     count slots (an item has < 2^16 tokens, words < 65535), spilling to the
+//     global (file, word) table when a probe run is exhausted;
+//   - at the item's end a whole-file item writes its records straight into
+//     the caller's array (one atomic per item reserves the space); chunks of
+//     larger files merge through the (file, word) table.
+constexpr uint32_t kWStep = 1024;            // bytes per warp step
+constexpr uint32_t kWBuf = kWStep + 64;      // + lookahead (a token starting in the step reads <= 48 past it)
+constexpr uint32_t kWTok = kWStep / 2;       // token starts per step at most
+constexpr uint32_t kWProbe = 32;             // count-table probe run before a spill
+struct WarpSmemLayout {
+  static __host__ __device__ constexpr uint32_t buf() { return 0; }
+  static __host__ __device__ constexpr uint32_t mask() { return kWBuf + 16; }
+  static __host__ __device__ constexpr uint32_t tok() { return mask() + 36 * 4; }
+  static __host__ __device__ constexpr uint32_t tab() { return tok() + kWTok * 2; }
+  static __host__ __device__ constexpr uint32_t bytes(uint32_t slots) { return tab() + slots * 4; }
+};
+
+__device__ __forceinline__ uint32_t word_bits32_regs(uint4 a, uint4 b) {
+  return word_bits4(a.x) | (word_bits4(a.y) << 4) | (word_bits4(a.z) << 8) | (word_bits4(a.w) << 12) |
+         (word_bits4(b.x) << 16) | (word_bits4(b.y) << 20) | (word_bits4(b.z) << 24) | (word_bits4(b.w) << 28);
+}
+__device__ __forceinline__ uint32_t lds_u32(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(detail::smem_u32(p)) : "memory");
+  return v;
+}
+__device__ __forceinline__ uint32_t atoms_cas32(uint32_t* p, uint32_t cmp, uint32_t v) {
+  uint32_t r;
+  asm volatile("atom.shared.cas.b32 %0, [%1], %2, %3;" : "=r"(r) : "r"(detail::smem_u32(p)), "r"(cmp), "r"(v)
+               : "memory");
+  return r;
+}
+__device__ __forceinline__ void reds_add32(uint32_t* p, uint32_t v) {
+  asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(detail::smem_u32(p)), "r"(v) : "memory");
+}
+
+// One hit of word k in the warp's count table; false when the probe run is
+// exhausted (the caller spills the hit to the (file, word) table).
+__device__ __forceinline__ bool wcount(uint32_t* tab, uint32_t tmask, uint32_t k) {
+  const uint32_t key = (k + 1) << 16;
+  uint32_t s = (k * 2654435761u) & tmask;
+  for (uint32_t p = 0; p < kWProbe; ++p, s = (s + 1) & tmask) {
+    uint32_t v = lds_u32(&tab[s]);
+    if (v == 0) {
+      v = atoms_cas32(&tab[s], 0u, key | 1u);
+      if (v == 0) return true;
+    }
+    if ((v & 0xFFFF0000u) == key) {
+      reds_add32(&tab[s], 1u);
+      return true;
+    }
+  }
+  return false;
+}
+
+struct WHit {
+  uint64_t dsum, dxor, nh;
+  uint32_t spilled;
+};
+__device__ __forceinline__ void whit(const GrepWork& w, uint32_t* tab, uint32_t tmask, uint32_t f, uint64_t hf,
+                                     uint32_t k, uint64_t pos, uint64_t* hits, uint64_t hit_cap, WHit& a) {
+  if (!wcount(tab, tmask, k)) {
+    pair_add(w, f, k, 1);  // this item's records then all go through the global table
+    a.spilled = 1;
+  }
+  const uint64_t m = hit_mix_hf(hf, pos, k);
+  a.dsum += m;
+  a.dxor ^= m;
+  ++a.nh;
+  if (hits) hit_list(w, f, k, pos, hits, hit_cap);
+}
+
+// The token's bytes buf[i, i + L) as 8 zero-padded words.
+__device__ __forceinline__ void wtoken_words(const uint8_t* buf, uint32_t i, uint32_t L, uint32_t (&v)[8]) {
+  uint32_t W[12];
+  const uint4* qv = (const uint4*)(buf + (i & ~15u));
+#pragma unroll
+  for (int j = 0; j < 3; ++j) {
+    const uint4 t = qv[j];
+    W[4 * j] = t.x;
+    W[4 * j + 1] = t.y;
+    W[4 * j + 2] = t.z;
+    W[4 * j + 3] = t.w;
+  }
+  gather_token(W, i & 15u, L, v);
+}
+__device__ __forceinline__ bool wsame(const GrepWork& w, uint32_t kp, const uint32_t (&v)[8]) {
+  const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
+  const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
+  return ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) | (d1.y ^ v[5]) |
+          (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
+}
+// A hit of table entry `ent` (word kp, and its duplicates, R14).
+__device__ __forceinline__ void whit_entry(const GrepWork& w, uint32_t* tab, uint32_t tmask, uint32_t f, uint64_t hf,
+                                           uint64_t ent, uint64_t pos, uint64_t* hits, uint64_t hit_cap, WHit& a) {
+  const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
+  whit(w, tab, tmask, f, hf, kp, pos, hits, hit_cap, a);
+  if (ent & kDupBit)
+    for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1]) whit(w, tab, tmask, f, hf, d - 1, pos, hits, hit_cap, a);
+}
+// One token buf[i, i + L) (1 <= L <= 32) at file position pos: hash, L1
+// filter, one 32-byte bucket of the table per step, an exact compare on a key
+// match (as scan_token).
+__device__ __forceinline__ void wscan_token(const GrepWork& w, const uint8_t* buf, uint32_t* tab, uint32_t tmask,
+                                            uint32_t f, uint64_t hf, uint32_t i, uint32_t L, uint64_t pos,
+                                            uint64_t* hits, uint64_t hit_cap, WHit& a) {
+  const uint32_t* q = (const uint32_t*)(buf + (i & ~3u));
+  const uint32_t a0 = q[0], a1 = q[1], a2 = q[2], r8 = (i & 3u) * 8;
+  const uint32_t w0 = low_bytes(__funnelshift_r(a0, a1, r8), min((int)L, 4));
+  const uint32_t w1 = low_bytes(__funnelshift_r(a1, a2, r8), min(max((int)L - 4, 0), 4));
+  const uint64_t h = tok_hash(w0, w1, L);
+  const uint32_t fi = filter_index(h, w.filt_log2);
+  if (!((ld_filter(&w.filt[fi >> 5]) >> (fi & 31)) & 1u)) return;
+  const uint64_t want = entry_key(h, L) >> 26;
+  uint32_t b = (uint32_t)h & w.table_mask & ~3u;
+  for (;;) {
+    const uint4* bp = (const uint4*)&w.table[b];
+    const uint4 e01 = __ldg(bp), e23 = __ldg(bp + 1);
+    const uint64_t ent[4] = {((uint64_t)e01.y << 32) | e01.x, ((uint64_t)e01.w << 32) | e01.z,
+                             ((uint64_t)e23.y << 32) | e23.x, ((uint64_t)e23.w << 32) | e23.z};
+    bool empty = false;
+#pragma unroll
+    for (int e = 0; e < 4; ++e) {
+      empty |= ent[e] == 0;
+      if (ent[e] != 0 && key_bits(ent[e]) == want) {
+        uint32_t v[8];
+        wtoken_words(buf, i, L, v);
+        if (wsame(w, (uint32_t)(ent[e] & ((1u << 26) - 1)) - 1, v)) {
+          whit_entry(w, tab, tmask, f, hf, ent[e], pos, hits, hit_cap, a);
+          return;
+        }
+      }
+    }
+    if (empty) return;
+    b = (b + 4) & w.table_mask;
+  }
+}
+
+// 32 bytes of lane `lane` of the step at p (a 1 KiB-aligned frame address);
+// zeros for lanes >= nl.
+__device__ __forceinline__ void wload(const uint8_t* p, int lane, int nl, uint4& a, uint4& b) {
+  if (p && lane < nl) {
+    const uint4* q = (const uint4*)(p + 32 * lane);
+    a = __ldcs(q);  // streamed: the step is read once (its bytes are staged in shared memory)
+    b = __ldcs(q + 1);
+  } else {
+    a = make_uint4(0, 0, 0, 0);
+    b = a;
+  }
+}
+
+// gmmap_warp of one whole page, out of line (once per page: the scan loop
+// keeps its registers and the kernel its instruction cache footprint).
+__device__ __noinline__ const uint8_t* wmap_page(const gfs_ctx* c, int fd, uint64_t q, int* err) {
+  uint64_t m = 0;
+  return (const uint8_t*)gmmap_t<detail::WarpGroup>(c, nullptr, c->page_size, 0, 0, fd, q << c->page_shift, &m, err);
+}
+__device__ __noinline__ void wunmap_page(const gfs_ctx* c, const uint8_t* p) { gmunmap_warp(c, (void*)p, 1); }
+
+// A warp's two most recent page mappings (gmmap_warp); pages only advance, so
+// mapping a new page releases the older one. Warp-uniform.
+struct WPageWin {
+  uint64_t pg0 = ~0ull, pg1 = ~0ull;
+  const uint8_t* pp0 = nullptr;
+  const uint8_t* pp1 = nullptr;
+  int err = 0;
+  __device__ __forceinline__ const uint8_t* map(const gfs_ctx* c, int fd, uint64_t q) {
+    if (pg0 == q) return pp0;
+    if (pg1 == q) return pp1;
+    if (err) return nullptr;
+    const bool use0 = pg0 == ~0ull || (pg1 != ~0ull && pg0 < pg1);
+    const uint8_t* old = use0 ? pp0 : pp1;
+    if (old) wunmap_page(c, old);
+    int er = 0;
+    const uint8_t* p = wmap_page(c, fd, q, &er);
+    if (!p) err = er ? er : -EIO;
+    if (use0) {
+      pg0 = p ? q : ~0ull;
+      pp0 = p;
+    } else {
+      pg1 = p ? q : ~0ull;
+      pp1 = p;
+    }
+    return p;
+  }
+  __device__ __forceinline__ void release(const gfs_ctx* c) {
+    if (pp0) wunmap_page(c, pp0);
+    if (pp1) wunmap_page(c, pp1);
+  }
+};
+
+__global__ void __launch_bounds__(256) k_grep_wscan(const gfs_ctx* c, const __grid_constant__ GrepWork w,
+                                                    uint64_t* hits, uint64_t hit_cap, uint64_t* totals,
+                                                    uint32_t* rec, uint64_t rec_cap) {
+  extern __shared__ __align__(16) uint8_t sm[];
+  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+  const uint32_t slots = w.cslots, tmask = slots - 1;
+  uint8_t* ws = sm + (size_t)wid * WarpSmemLayout::bytes(slots);
+  uint8_t* buf = ws + WarpSmemLayout::buf();
+  uint32_t* msk = (uint32_t*)(ws + WarpSmemLayout::mask());
+  uint16_t* tok = (uint16_t*)(ws + WarpSmemLayout::tok());
+  uint32_t* tab = (uint32_t*)(ws + WarpSmemLayout::tab());
+  const uint32_t shift = c->page_shift;
+  const uint64_t P = c->page_size;
+  for (uint32_t i = lane; i < slots; i += 32) tab[i] = 0;  // dynamic smem is not cleared between launches
+  uint64_t nitems = count_items(w);
+  if (nitems > w.max_items) {
+    if (blockIdx.x == 0 && threadIdx.x == 0) set_err(w, -ENOSPC);
+    nitems = w.max_items;
+  }
+  if (blockIdx.x == 0 && threadIdx.x == 0) w.vars[V_NITEMS] = nitems;
+  WHit acc{0, 0, 0, 0};
+  unsigned long long it = 0;
+  if (lane == 0) it = atomicAdd(&w.vars[V_NEXT], 1ull);
+  it = __shfl_sync(0xFFFFFFFFu, it, 0);
+  while (it < nitems) {
+    const ItemDesc d = w.desc[it];
+    unsigned long long nxt = 0;
+    if (lane == 0) nxt = atomicAdd(&w.vars[V_NEXT], 1ull);  // the next item's claim flies meanwhile
+    const uint32_t f = d.gid;
+    const uint64_t hf = splitmix64(f);
+    const bool whole = d.meta >> 31;
+    const int fd = d.fd;
+    // token starts counted in [s, e); bytes read [s - 1, min(S, e + 33))
+    uint64_t s, e, S;
+    if (whole) {
+      s = 0;
+      e = S = d.rlen;
+    } else {
+      s = d.roff + (d.meta & 31u);
+      e = s + d.body;
+      S = w.size[d.f];
+    }
+    const uint64_t need_end = min(S, e + 33);
+    // two-page window of gmmap_warp mappings (pages only ever advance)
+    WPageWin pw;
+    uint32_t prev = 0;  // W(t[x - 1]) for the current step x
+    if (s > 0) {
+      const uint8_t* p = pw.map(c, fd, (s - 1) >> shift);
+      if (p) prev = is_word(p[(s - 1) & (P - 1)]) ? 1u : 0u;  // the same byte in every lane
+    }
+    uint64_t x = s;
+    uint4 ca, cb, na, nb;
+    {
+      const uint8_t* p = pw.map(c, fd, x >> shift);
+      wload(p ? p + (x & (P - 1)) : nullptr, lane, 32, ca, cb);
+    }
+    while (!pw.err && x < e) {
+      const uint64_t nx = x + kWStep;
+      // the next step: all of it if tokens start there, else the lookahead lanes
+      const uint8_t* np = nullptr;
+      int nl = 0;
+      if (nx < need_end) {
+        np = pw.map(c, fd, nx >> shift);
+        nl = nx < e ? 32 : 2;
+      }
+      wload(np ? np + (nx & (P - 1)) : nullptr, lane, nl, na, nb);
+      if (pw.err) break;
+      // stage this step (+ the next step's first 64 bytes) for the token gathers
+      *(uint4*)(buf + 32 * lane) = ca;
+      *(uint4*)(buf + 32 * lane + 16) = cb;
+      // word-byte masks; bytes at or past EOF are non-word
+      const uint64_t lb = x + 32 * (uint64_t)lane;
+      uint32_t m = word_bits32_regs(ca, cb);
+      if (lb + 32 > S) m &= lb >= S ? 0u : ((1u << (uint32_t)(S - lb)) - 1u);
+      msk[lane] = m;
+      if (lane < 2) {
+        *(uint4*)(buf + kWStep + 32 * lane) = na;
+        *(uint4*)(buf + kWStep + 32 * lane + 16) = nb;
+        const uint64_t lnb = nx + 32 * (uint64_t)lane;
+        uint32_t mn = word_bits32_regs(na, nb);
+        if (lnb + 32 > S) mn &= lnb >= S ? 0u : ((1u << (uint32_t)(S - lnb)) - 1u);
+        msk[32 + lane] = mn;
+      }
+      // token starts in [x, e): W(t[i]) and not W(t[i - 1])
+      const uint32_t up = __shfl_up_sync(0xFFFFFFFFu, m, 1);
+      const uint32_t pl = lane ? (up >> 31) : prev;
+      uint32_t st = m & ~((m << 1) | pl);
+      if (lb + 32 > e) st &= lb >= e ? 0u : ((1u << (uint32_t)(e - lb)) - 1u);
+      prev = __shfl_sync(0xFFFFFFFFu, m, 31) >> 31;
+      const uint32_t cnt = __popc(st);
+      uint32_t incl = cnt;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, incl, o);
+        if (lane >= o) incl += t;
+      }
+      const uint32_t total = __shfl_sync(0xFFFFFFFFu, incl, 31);
+      uint32_t o = incl - cnt;
+      for (uint32_t y = st; y; y &= y - 1) tok[o++] = (uint16_t)(32 * lane + __ffs(y) - 1);
+      __syncwarp();
+      for (uint32_t q = lane; q < total; q += 32) {
+        const uint32_t i = tok[q], j = i >> 5, b = i & 31;
+        const uint64_t win = ((uint64_t)msk[j + 1] << 32) | msk[j];
+        const uint32_t L = __ffsll(~(win >> b)) - 1;  // >= 33: too long for any word (R12)
+        if (L <= 32) wscan_token(w, buf, tab, tmask, f, hf, i, L, x + i, hits, hit_cap, acc);
+      }
+      __syncwarp();  // buf / msk / tok are rewritten by the next step
+      ca = na;
+      cb = nb;
+      x = nx;
+    }
+    pw.release(c);
+    const int err = pw.err;
+    if (err && lane == 0) set_err(w, err);
+    // flush: the warp's occupied slots -> records (direct) or the (file, word) table
+    const bool direct = whole && !__any_sync(0xFFFFFFFFu, acc.spilled) && rec && !err;
+    acc.spilled = 0;
+    uint32_t nocc = 0;
+    for (uint32_t i = lane; i < slots; i += 32) nocc += tab[i] != 0;
+    unsigned long long base = 0;
+    if (direct) {
+      uint32_t inc = nocc;
+#pragma unroll
+      for (int o2 = 1; o2 < 32; o2 <<= 1) {
+        const uint32_t t = __shfl_up_sync(0xFFFFFFFFu, inc, o2);
+        if (lane >= o2) inc += t;
+      }
+      const uint32_t all = __shfl_sync(0xFFFFFFFFu, inc, 31);
+      if (lane == 31 && all) base = atomicAdd(&w.vars[V_NDIRECT], (unsigned long long)all);
+      base = __shfl_sync(0xFFFFFFFFu, base, 31) + (inc - nocc);
+    }
+    for (uint32_t i = lane; i < slots; i += 32) {
+      const uint32_t v = tab[i];
+      if (!v) continue;
+      tab[i] = 0;
+      if (err) continue;
+      const uint32_t k = (v >> 16) - 1, n = v & 0xFFFFu;
+      if (direct) {
+        atomicAdd((unsigned long long*)&totals[k], (unsigned long long)n);
+        if (base < rec_cap) {
+          uint32_t* r = rec + 3 * base;
+          r[0] = f;
+          r[1] = k;
+          r[2] = n;
+        }
+        ++base;
+      } else {
+        pair_add(w, f, k, n);
+      }
+    }
+    __syncwarp();
+    it = __shfl_sync(0xFFFFFFFFu, nxt, 0);
+  }
+  for (int o = 16; o; o >>= 1) {
+    acc.dsum += __shfl_xor_sync(0xFFFFFFFFu, acc.dsum, o);
+    acc.dxor ^= __shfl_xor_sync(0xFFFFFFFFu, acc.dxor, o);
+    acc.nh += __shfl_xor_sync(0xFFFFFFFFu, acc.nh, o);
+  }
+  if (lane == 0) {
+    atomicAdd(&w.vars[V_DSUM], (unsigned long long)acc.dsum);
+    atomicXor(&w.vars[V_DXOR], (unsigned long long)acc.dxor);
+    atomicAdd(&w.vars[V_NHITS], (unsigned long long)acc.nh);
+  }
+}
+
 __global__ void k_grep_close(const gfs_ctx* c, const __grid_constant__ GrepWork w) {
   const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
   for (uint32_t f = blockIdx.x; f < nfiles; f += gridDim.x) {
@@ -1161,7 +1532,7 @@ __global__ void k_grep_pack_scan(const __grid_constant__ GrepWork w, uint64_t re
   part[tid] = s;
   __syncthreads();
   if (tid == 0) {
-    uint64_t run = 0;
+    uint64_t run = w.vars[V_NDIRECT];  // the warp scan's direct records come first
     for (uint32_t q = 0; q < nthr; ++q) {
       const uint64_t v = part[q];
       part[q] = run;
@@ -1280,6 +1651,19 @@ uint32_t pick_cslots(uint32_t chunk, uint32_t block) {
   return cs;
 }
 
+// Count-table slots per warp of the warp scan (a power of two; GFS_GREP_WSLOTS
+// overrides it for tuning): 1024 hold the ~560 distinct words of a 32 KiB C4
+// item at about half load and leave room for 24 warps per SM (2048 with 64 KiB
+// items: 16 warps per SM, measured slower).
+uint32_t wscan_slots() {
+  uint32_t v = 1024;
+  if (const char* e = getenv("GFS_GREP_WSLOTS")) {
+    const long x = atol(e);
+    if (x >= 256 && x <= 8192 && (x & (x - 1)) == 0) v = (uint32_t)x;
+  }
+  return v;
+}
+
 }  // namespace
 
 GFS_API uint64_t gfs_grep_work_bytes(const gfs_grep_params* p) { return p ? layout(p).total : 0; }
@@ -1289,8 +1673,13 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
                      uint64_t* d_hits, uint64_t* d_summary) {
   if (!h || !dict_path || !list_path || !p || !d_work || !d_totals || !d_summary || p->max_files == 0 ||
       p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) ||
-      p->chunk + kPre + kHalo > 65536 ||  // 16-bit token offsets into the item buffer
-      p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31))
+      p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31) || p->scan > 1)
+    return -EINVAL;
+  const bool wscan = p->scan == 1;
+  if (!wscan && p->chunk + kPre + kHalo > 65536) return -EINVAL;  // 16-bit token offsets into the item buffer
+  // warp scan: 1 KiB steps never straddle a chunk; an item has < 2^16 tokens
+  // and a word index fits the 16-bit key of a count slot
+  if (wscan && ((p->chunk & (kWStep - 1)) || p->chunk > 65536 || p->whole_max > 65536 || p->max_words >= 65535))
     return -EINVAL;
   cudaStream_t s = (cudaStream_t)stream;
   const Layout L = layout(p);
@@ -1310,8 +1699,14 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   w.desc = (ItemDesc*)(base + L.off[9]);
   w.max_items = L.max_items;
   w.chunk = p->chunk;
-  w.cslots = pick_cslots(p->chunk, p->block);
-  {
+  w.cslots = wscan ? wscan_slots() : pick_cslots(p->chunk, p->block);
+  if (wscan) {
+    // whole-file items up to whole_max (default: 2 chunks), counted by one warp
+    const uint32_t wm = p->whole_max ? p->whole_max : 2 * p->chunk;
+    const uint32_t wc = wm / p->chunk;
+    w.whole_chunks = wc < kMaxWholeChunks ? wc : kMaxWholeChunks;
+    if ((uint64_t)w.whole_chunks * p->chunk > 65536) w.whole_chunks = 65536 / p->chunk;
+  } else {
     // default: what the count table holds (~64 text bytes per distinct word)
     const uint32_t wm = p->whole_max ? p->whole_max : w.cslots * 64u;
     const uint32_t wc = wm / p->chunk;
@@ -1350,9 +1745,10 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
     if (d_prof) cudaMemsetAsync(d_prof, 0, 8 * sizeof(unsigned long long), s);
     w.prof = d_prof;
   }
-  const uint32_t smem = scan_smem(p->chunk, p->block, w.cslots);
-  if (smem > 227 * 1024) return -EINVAL;
-  cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  const uint32_t smem = wscan ? (p->block / 32) * WarpSmemLayout::bytes(w.cslots) : scan_smem(p->chunk, p->block, w.cslots);
+  if (smem > 200 * 1024) return -EINVAL;
+  if (wscan) cudaFuncSetAttribute(k_grep_wscan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  else cudaFuncSetAttribute(k_grep_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   int dev = 0, nsm = 148;
   cudaGetDevice(&dev);
   cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, dev);
@@ -1376,10 +1772,15 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
   // persistent scan grid: every resident block slot once (p->grid caps it)
   int occ = 1;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_scan, (int)p->block, smem);
+  if (wscan) cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_wscan, (int)p->block, smem);
+  else cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_grep_scan, (int)p->block, smem);
   const uint32_t scan_grid = (uint32_t)(occ > 0 ? occ : 1) * (uint32_t)nsm;
-  k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
-      c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
+  if (wscan)
+    k_grep_wscan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
+        c, w, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
+  else
+    k_grep_scan<<<scan_grid < p->grid ? scan_grid : p->grid, p->block, smem, s>>>(
+        c, w, p->chunk, d_hits, d_hits ? p->hit_cap : 0, d_totals, d_rec, d_rec ? rec_cap : 0);
   if (!p->keep_open) k_grep_close<<<nsm * 16, 32, 0, s>>>(c, w);
   k_grep_compact<<<nsm * 4, 256, 0, s>>>(w, d_rec ? 1 : 0, d_totals);
   if (d_rec) {
