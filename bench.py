@@ -649,7 +649,10 @@ def matvec_phase(X, h2d):
                 zy = state["y"].cpu().numpy()
             out["zero_copy"] = {"GBps": round(gbs(nbytes, zt[0]), 3), "frac_h2d": round(gbs(nbytes, zt[0]) / h2d, 4),
                                 "register_s": round(reg_s, 2), "zc_fill": zst["zc_fill"], "rpc_read": zst["rpc_read"],
-                                "path_used": zst["zc_fill"] > 0 and zst["rpc_read"] == 0,
+                                # every matrix page through the registered mapping; the only READ RPCs are
+                                # the x vector's pages (x is not registered)
+                                "path_used": (zst["zc_fill"] >= -(-nbytes // (2 << 20))
+                                              and zst["rpc_read"] <= -(-cols * 4 // (2 << 20))),
                                 "y_equal_rpc_path": bool(np.array_equal(zy, ymine))}
         except Exception as e:
             out["zero_copy"] = {"unavailable": str(e)[:200]}
@@ -1188,9 +1191,10 @@ def main():
     ap.add_argument("--reps", type=int, default=5, help="timed repetitions of the secondary phases (mean, stddev)")
     ap.add_argument("--hit-file-gib", type=int, default=4)
     ap.add_argument("--hit-page-kib", type=int, default=512)
-    ap.add_argument("--hit-grid", type=int, default=1184)   # 8 blocks/SM: lookups of one block overlap
-    ap.add_argument("--hit-block", type=int, default=128)   # copies of the others (measured best)
-    ap.add_argument("--hit-calls", type=int, default=1024)
+    ap.add_argument("--hit-grid", type=int, default=1480)   # 10 blocks/SM (the register limit at 96 threads):
+    ap.add_argument("--hit-block", type=int, default=96)    # lookups of one block overlap copies of the others
+                                                            # (tools/k4_occ.py: 96 x 10 measured best)
+    ap.add_argument("--hit-calls", type=int, default=820)  # ~1.21 M calls in all (1184 x 1024 before)
     ap.add_argument("--hg-gib", type=int, default=16, help="hit->global file size (GiB)")
     ap.add_argument("--hg-grid", type=int, default=592)
     ap.add_argument("--ref-sample-mib", type=int, default=2048)
