@@ -786,6 +786,45 @@ __device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, 
   if (hits) hit_list(w, f, k, pos, hits, hit_cap);
 }
 
+// The next table entry at or after (bucket b, entry q) whose key (fingerprint
+// + length) is `want`: returns it and advances (b, q) past it, or returns 0
+// at the first empty entry (insertion filled the first empty slot in probe
+// order and nothing is ever removed, so an empty slot ends the search). The
+// caller verifies a candidate with ONE copy of its compare-and-count code
+// (a match found in entry 0..3 of a bucket takes the same path: no warp
+// divergence on the entry position).
+__device__ __forceinline__ uint64_t next_candidate(const GrepWork& w, uint64_t want, uint32_t& b, uint32_t& q) {
+  for (;;) {
+    const uint4* bp = (const uint4*)&w.table[b];
+    const uint4 e01 = __ldg(bp), e23 = __ldg(bp + 1);
+    const uint64_t ent[4] = {((uint64_t)e01.y << 32) | e01.x, ((uint64_t)e01.w << 32) | e01.z,
+                             ((uint64_t)e23.y << 32) | e23.x, ((uint64_t)e23.w << 32) | e23.z};
+    uint64_t cand = 0;
+    uint32_t cq = 4;
+    bool empty = false;
+#pragma unroll
+    for (uint32_t e = 0; e < 4; ++e) {
+      const bool look = e >= q && cq == 4 && !empty;
+      if (look && ent[e] == 0) empty = true;
+      else if (look && key_bits(ent[e]) == want) {
+        cand = ent[e];
+        cq = e;
+      }
+    }
+    if (cq < 4) {
+      q = cq + 1;
+      if (q == 4) {
+        q = 0;
+        b = (b + 4) & w.table_mask;
+      }
+      return cand;
+    }
+    if (empty) return 0;
+    q = 0;
+    b = (b + 4) & w.table_mask;
+  }
+}
+
 // One token: bytes buf[i, i + L), file position pos, 1 <= L <= 32.
 __device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S, uint32_t* spilled,
                                            uint32_t f, uint32_t i, uint32_t L, uint64_t pos, uint64_t* hits,
@@ -799,50 +838,37 @@ __device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S,
   const uint32_t fi = filter_index(h, w.filt_log2);
   if (!((ld_filter(&w.filt[fi >> 5]) >> (fi & 31)) & 1u)) return;
   const uint64_t want = entry_key(h, L) >> 26;
-  // One 32-byte bucket (4 entries) per step; insertion filled the first empty
-  // slot in the same order, so an empty slot ends the search.
-  uint32_t b = (uint32_t)h & w.table_mask & ~3u;
+  uint32_t b = (uint32_t)h & w.table_mask & ~3u, q = 0;
   for (;;) {
-    const uint4* bp = (const uint4*)&w.table[b];
-    const uint4 e01 = __ldg(bp), e23 = __ldg(bp + 1);
-    const uint64_t ent[4] = {((uint64_t)e01.y << 32) | e01.x, ((uint64_t)e01.w << 32) | e01.z,
-                             ((uint64_t)e23.y << 32) | e23.x, ((uint64_t)e23.w << 32) | e23.z};
-    bool empty = false;
+    const uint64_t ent = next_candidate(w, want, b, q);
+    if (!ent) return;
+    const uint32_t kp = (uint32_t)(ent & ((1u << 26) - 1)) - 1;
+    const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
+    const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
+    uint32_t v[8];  // the whole token, zero-padded: only gathered on a key match
+    {
+      uint32_t W[12];
+      const uint4* qv = (const uint4*)(S.buf + (i & ~15u));
 #pragma unroll
-    for (int q = 0; q < 4; ++q) {
-      empty |= ent[q] == 0;
-      if (ent[q] != 0 && key_bits(ent[q]) == want) {
-        const uint32_t kp = (uint32_t)(ent[q] & ((1u << 26) - 1)) - 1;
-        const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
-        const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
-        uint32_t v[8];  // the whole token, zero-padded: only gathered on a key match
-        {
-          uint32_t W[12];
-          const uint4* qv = (const uint4*)(S.buf + (i & ~15u));
-#pragma unroll
-          for (int j = 0; j < 3; ++j) {
-            const uint4 t = qv[j];
-            W[4 * j] = t.x;
-            W[4 * j + 1] = t.y;
-            W[4 * j + 2] = t.z;
-            W[4 * j + 3] = t.w;
-          }
-          gather_token(W, i & 15u, L, v);
-        }
-        const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
-                           (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
-        if (same) {
-          count_hit(w, S, spilled, f, kp, pos, hits, hit_cap, acc);
-          if (ent[q] & kDupBit) {  // the word's duplicates each count (R14)
-            for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
-              count_hit(w, S, spilled, f, d - 1, pos, hits, hit_cap, acc);
-          }
-          return;
-        }
+      for (int j = 0; j < 3; ++j) {
+        const uint4 t = qv[j];
+        W[4 * j] = t.x;
+        W[4 * j + 1] = t.y;
+        W[4 * j + 2] = t.z;
+        W[4 * j + 3] = t.w;
       }
+      gather_token(W, i & 15u, L, v);
     }
-    if (empty) return;
-    b = (b + 4) & w.table_mask;
+    const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
+                       (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
+    if (same) {
+      count_hit(w, S, spilled, f, kp, pos, hits, hit_cap, acc);
+      if (ent & kDupBit) {  // the word's duplicates each count (R14)
+        for (uint32_t d = w.dup_head[kp]; d; d = w.dup_next[d - 1])
+          count_hit(w, S, spilled, f, d - 1, pos, hits, hit_cap, acc);
+      }
+      return;
+    }
   }
 }
 
@@ -1198,35 +1224,24 @@ __device__ __forceinline__ void whit_entry(const GrepWork& w, uint32_t* tab, uin
 __device__ __forceinline__ void wscan_token(const GrepWork& w, const uint8_t* buf, uint32_t* tab, uint32_t tmask,
                                             uint32_t f, uint64_t hf, uint32_t i, uint32_t L, uint64_t pos,
                                             uint64_t* hits, uint64_t hit_cap, WHit& a) {
-  const uint32_t* q = (const uint32_t*)(buf + (i & ~3u));
-  const uint32_t a0 = q[0], a1 = q[1], a2 = q[2], r8 = (i & 3u) * 8;
+  const uint32_t* qw = (const uint32_t*)(buf + (i & ~3u));
+  const uint32_t a0 = qw[0], a1 = qw[1], a2 = qw[2], r8 = (i & 3u) * 8;
   const uint32_t w0 = low_bytes(__funnelshift_r(a0, a1, r8), min((int)L, 4));
   const uint32_t w1 = low_bytes(__funnelshift_r(a1, a2, r8), min(max((int)L - 4, 0), 4));
   const uint64_t h = tok_hash(w0, w1, L);
   const uint32_t fi = filter_index(h, w.filt_log2);
   if (!((ld_filter(&w.filt[fi >> 5]) >> (fi & 31)) & 1u)) return;
   const uint64_t want = entry_key(h, L) >> 26;
-  uint32_t b = (uint32_t)h & w.table_mask & ~3u;
+  uint32_t b = (uint32_t)h & w.table_mask & ~3u, q = 0;
   for (;;) {
-    const uint4* bp = (const uint4*)&w.table[b];
-    const uint4 e01 = __ldg(bp), e23 = __ldg(bp + 1);
-    const uint64_t ent[4] = {((uint64_t)e01.y << 32) | e01.x, ((uint64_t)e01.w << 32) | e01.z,
-                             ((uint64_t)e23.y << 32) | e23.x, ((uint64_t)e23.w << 32) | e23.z};
-    bool empty = false;
-#pragma unroll
-    for (int e = 0; e < 4; ++e) {
-      empty |= ent[e] == 0;
-      if (ent[e] != 0 && key_bits(ent[e]) == want) {
-        uint32_t v[8];
-        wtoken_words(buf, i, L, v);
-        if (wsame(w, (uint32_t)(ent[e] & ((1u << 26) - 1)) - 1, v)) {
-          whit_entry(w, tab, tmask, f, hf, ent[e], pos, hits, hit_cap, a);
-          return;
-        }
-      }
+    const uint64_t ent = next_candidate(w, want, b, q);
+    if (!ent) return;
+    uint32_t v[8];
+    wtoken_words(buf, i, L, v);
+    if (wsame(w, (uint32_t)(ent & ((1u << 26) - 1)) - 1, v)) {
+      whit_entry(w, tab, tmask, f, hf, ent, pos, hits, hit_cap, a);
+      return;
     }
-    if (empty) return;
-    b = (b + 4) & w.table_mask;
   }
 }
 

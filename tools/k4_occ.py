@@ -34,7 +34,7 @@ with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, daemon_threads=12) as 
     assert fs.seqread(path, size, P, grid=296)[1] == 0
     raw = torch.empty(size, dtype=torch.uint8, device=dev)
     raw.copy_(torch.from_file(path, shared=False, size=size, dtype=torch.uint8))
-    for block, per_sm in [(128, 8), (64, 8), (64, 10), (64, 12), (32, 12), (96, 10)]:
+    for block, per_sm in [(128, 8), (96, 10), (64, 12)]:
         grid = 148 * per_sm
         calls = total_calls // grid
         rng = np.random.default_rng(7)
