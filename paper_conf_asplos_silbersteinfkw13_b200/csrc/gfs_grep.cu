@@ -179,20 +179,19 @@ __device__ __forceinline__ uint32_t low_bytes(uint32_t x, int nb) {
   return x & __funnelshift_lc(0xFFFFFFFFu, 0u, 8 * nb);
 }
 
-// Bytes [0, L) of the 32 starting at byte offset `sh` (0..15) of 12 words,
-// as 8 zero-padded words: two select levels + a funnel shift, no local memory.
-__device__ __forceinline__ void gather_token(const uint32_t (&W)[12], uint32_t sh, uint32_t L, uint32_t (&v)[8]) {
-  uint32_t A[10], B[9];
+// Bytes [i, i + L) of buf (4-byte aligned shared memory, >= 36 readable
+// bytes from i & ~3) as 8 zero-padded words: nine word loads and funnel
+// shifts (no select chains).
+__device__ __forceinline__ void token_words(const uint8_t* buf, uint32_t i, uint32_t L, uint32_t (&v)[8]) {
+  const uint32_t* q = (const uint32_t*)(buf + (i & ~3u));
+  const uint32_t r = (i & 3u) * 8;
+  uint32_t wv[9];
 #pragma unroll
-  for (int j = 0; j < 10; ++j) A[j] = (sh & 8) ? W[j + 2] : W[j];
-#pragma unroll
-  for (int j = 0; j < 9; ++j) B[j] = (sh & 4) ? A[j + 1] : A[j];
-  const uint32_t r = (sh & 3) * 8;
+  for (int j = 0; j < 9; ++j) wv[j] = q[j];
 #pragma unroll
   for (int j = 0; j < 8; ++j) {
-    const uint32_t wv = __funnelshift_r(B[j], B[j + 1], r);
     const int nb = min(max((int)L - 4 * j, 0), 4);
-    v[j] = wv & __funnelshift_lc(0xFFFFFFFFu, 0u, 8 * nb);  // low nb bytes
+    v[j] = __funnelshift_r(wv[j], wv[j + 1], r) & __funnelshift_lc(0xFFFFFFFFu, 0u, 8 * nb);
   }
 }
 
@@ -747,6 +746,11 @@ __device__ __forceinline__ void reds_add(uint32_t* p, uint32_t v) {
 __device__ __forceinline__ void reds_or(uint32_t* p, uint32_t v) {
   asm volatile("red.shared.or.b32 [%0], %1;" ::"r"(detail::smem_u32(p)), "r"(v) : "memory");
 }
+__device__ __forceinline__ uint32_t lds_u32(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(detail::smem_u32(p)) : "memory");
+  return v;
+}
 
 // The rare per-hit paths, out of line (the token loop keeps its registers).
 __device__ __noinline__ void hit_spill(const GrepWork& w, uint32_t f, uint32_t k, uint32_t* spilled) {
@@ -770,8 +774,11 @@ __device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, 
   uint32_t cs = (k * 2654435761u) & S.cmask;
   bool done = false;
   for (uint32_t p = 0; p < 64; ++p, cs = (cs + 1) & S.cmask) {
-    const uint32_t prev = atoms_cas(&S.ckey[cs], 0u, k + 1);
-    if (prev == 0) reds_or(&S.occ[cs >> 5], 1u << (cs & 31));
+    uint32_t prev = lds_u32(&S.ckey[cs]);  // a word seen before in this item: no atomic on the key
+    if (prev == 0) {
+      prev = atoms_cas(&S.ckey[cs], 0u, k + 1);
+      if (prev == 0) reds_or(&S.occ[cs >> 5], 1u << (cs & 31));
+    }
     if (prev == 0 || prev == k + 1) {
       reds_add(&S.ccnt[cs], 1u);
       done = true;
@@ -846,19 +853,7 @@ __device__ __forceinline__ void scan_token(const GrepWork& w, const ScanSmem& S,
     const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
     const uint4 d0 = __ldg(dw), d1 = __ldg(dw + 1);
     uint32_t v[8];  // the whole token, zero-padded: only gathered on a key match
-    {
-      uint32_t W[12];
-      const uint4* qv = (const uint4*)(S.buf + (i & ~15u));
-#pragma unroll
-      for (int j = 0; j < 3; ++j) {
-        const uint4 t = qv[j];
-        W[4 * j] = t.x;
-        W[4 * j + 1] = t.y;
-        W[4 * j + 2] = t.z;
-        W[4 * j + 3] = t.w;
-      }
-      gather_token(W, i & 15u, L, v);
-    }
+    token_words(S.buf, i, L, v);
     const bool same = ((d0.x ^ v[0]) | (d0.y ^ v[1]) | (d0.z ^ v[2]) | (d0.w ^ v[3]) | (d1.x ^ v[4]) |
                        (d1.y ^ v[5]) | (d1.z ^ v[6]) | (d1.w ^ v[7])) == 0;
     if (same) {
@@ -1139,11 +1134,6 @@ __device__ __forceinline__ uint32_t word_bits32_regs(uint4 a, uint4 b) {
   return word_bits4(a.x) | (word_bits4(a.y) << 4) | (word_bits4(a.z) << 8) | (word_bits4(a.w) << 12) |
          (word_bits4(b.x) << 16) | (word_bits4(b.y) << 20) | (word_bits4(b.z) << 24) | (word_bits4(b.w) << 28);
 }
-__device__ __forceinline__ uint32_t lds_u32(const uint32_t* p) {
-  uint32_t v;
-  asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(detail::smem_u32(p)) : "memory");
-  return v;
-}
 __device__ __forceinline__ uint32_t atoms_cas32(uint32_t* p, uint32_t cmp, uint32_t v) {
   uint32_t r;
   asm volatile("atom.shared.cas.b32 %0, [%1], %2, %3;" : "=r"(r) : "r"(detail::smem_u32(p)), "r"(cmp), "r"(v)
@@ -1192,17 +1182,7 @@ __device__ __forceinline__ void whit(const GrepWork& w, uint32_t* tab, uint32_t 
 
 // The token's bytes buf[i, i + L) as 8 zero-padded words.
 __device__ __forceinline__ void wtoken_words(const uint8_t* buf, uint32_t i, uint32_t L, uint32_t (&v)[8]) {
-  uint32_t W[12];
-  const uint4* qv = (const uint4*)(buf + (i & ~15u));
-#pragma unroll
-  for (int j = 0; j < 3; ++j) {
-    const uint4 t = qv[j];
-    W[4 * j] = t.x;
-    W[4 * j + 1] = t.y;
-    W[4 * j + 2] = t.z;
-    W[4 * j + 3] = t.w;
-  }
-  gather_token(W, i & 15u, L, v);
+  token_words(buf, i, L, v);
 }
 __device__ __forceinline__ bool wsame(const GrepWork& w, uint32_t kp, const uint32_t (&v)[8]) {
   const uint4* dw = (const uint4*)(w.dict + (size_t)kp * 32);  // padded slot (k_grep_dict)
