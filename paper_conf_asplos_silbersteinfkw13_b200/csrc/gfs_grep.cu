@@ -801,32 +801,33 @@ __device__ __forceinline__ void count_hit(const GrepWork& w, const ScanSmem& S, 
 // (a match found in entry 0..3 of a bucket takes the same path: no warp
 // divergence on the entry position).
 __device__ __forceinline__ uint64_t next_candidate(const GrepWork& w, uint64_t want, uint32_t& b, uint32_t& q) {
+  const uint32_t want_hi = (uint32_t)(want >> 6), want_len = (uint32_t)want & 63u;
   for (;;) {
     const uint4* bp = (const uint4*)&w.table[b];
     const uint4 e01 = __ldg(bp), e23 = __ldg(bp + 1);
-    const uint64_t ent[4] = {((uint64_t)e01.y << 32) | e01.x, ((uint64_t)e01.w << 32) | e01.z,
-                             ((uint64_t)e23.y << 32) | e23.x, ((uint64_t)e23.w << 32) | e23.z};
-    uint64_t cand = 0;
-    uint32_t cq = 4;
-    bool empty = false;
+    const uint32_t lo[4] = {e01.x, e01.z, e23.x, e23.z}, hi[4] = {e01.y, e01.w, e23.y, e23.w};
+    // 4-bit masks of key matches and of empty entries; the first of either at
+    // or after q decides (key_bits: fingerprint = hi & 0x7fffffff, length =
+    // lo bits 26..31; an empty entry is all zero)
+    uint32_t mm = 0, em = 0;
 #pragma unroll
-    for (uint32_t e = 0; e < 4; ++e) {
-      const bool look = e >= q && cq == 4 && !empty;
-      if (look && ent[e] == 0) empty = true;
-      else if (look && key_bits(ent[e]) == want) {
-        cand = ent[e];
-        cq = e;
-      }
+    for (int e = 0; e < 4; ++e) {
+      mm |= (uint32_t)((hi[e] & 0x7FFFFFFFu) == want_hi && (lo[e] >> 26) == want_len && (lo[e] | hi[e])) << e;
+      em |= (uint32_t)((lo[e] | hi[e]) == 0) << e;
     }
-    if (cq < 4) {
-      q = cq + 1;
+    const uint32_t sel = (mm | em) & (0xFu << q);
+    if (sel) {
+      const uint32_t e = __ffs(sel) - 1;
+      if ((em >> e) & 1u) return 0;
+      const uint64_t cand = ((uint64_t)(e & 2 ? (e & 1 ? hi[3] : hi[2]) : (e & 1 ? hi[1] : hi[0])) << 32) |
+                            (e & 2 ? (e & 1 ? lo[3] : lo[2]) : (e & 1 ? lo[1] : lo[0]));
+      q = e + 1;
       if (q == 4) {
         q = 0;
         b = (b + 4) & w.table_mask;
       }
       return cand;
     }
-    if (empty) return 0;
     q = 0;
     b = (b + 4) & w.table_mask;
   }
