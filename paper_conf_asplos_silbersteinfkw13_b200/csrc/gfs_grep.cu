@@ -242,8 +242,9 @@ __device__ __forceinline__ uint32_t gid_of(const GrepWork& w, uint32_t f) { retu
 // next opener re-validate the file with the host (close-to-open).
 // With keep_open the two stay open until the next run (which opens them
 // again, then drops the previous run's references), like the corpus files.
-__global__ void k_grep_hold(const gfs_ctx* c, const char* dict_path, const char* list_path, const __grid_constant__ GrepWork w, int release,
+__global__ void k_grep_hold(const __grid_constant__ gfs_ctx cv_, const char* dict_path, const char* list_path, const __grid_constant__ GrepWork w, int release,
                             int keep_open) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   if (!release) {
     const int a = gopen(c, dict_path, GFS_O_RDONLY);
     const int b = gopen(c, list_path, GFS_O_RDONLY);
@@ -300,7 +301,8 @@ __global__ void k_grep_pairclear(const __grid_constant__ GrepWork w) {
 }
 
 // --------------------------------------------------------------- dictionary
-__global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, const __grid_constant__ GrepWork w, uint32_t max_words) {
+__global__ void k_grep_dict(const __grid_constant__ gfs_ctx cv_, const char* dict_path, const __grid_constant__ GrepWork w, uint32_t max_words) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int tid = threadIdx.x;
   const int fd = gopen(c, dict_path, GFS_O_RDONLY);
   if (fd < 0) {
@@ -374,7 +376,8 @@ __global__ void k_grep_dict(const gfs_ctx* c, const char* dict_path, const __gri
 
 // --------------------------------------------------------------- file list
 // Pass 1: every block greads its 64 KiB pieces of the list file.
-__global__ void k_grep_list_read(const gfs_ctx* c, const char* list_path, const __grid_constant__ GrepWork w, uint64_t list_cap) {
+__global__ void k_grep_list_read(const __grid_constant__ gfs_ctx cv_, const char* list_path, const __grid_constant__ GrepWork w, uint64_t list_cap) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, list_path, GFS_O_RDONLY);
   if (fd < 0) {
     if (threadIdx.x == 0 && blockIdx.x == 0) set_err(w, fd);
@@ -490,8 +493,9 @@ __global__ void k_grep_list_emit(const __grid_constant__ GrepWork w, uint32_t ma
 // whole files by chunk count, the chunks of larger files.
 __device__ __forceinline__ uint64_t item_count(uint64_t size, uint32_t chunk) { return (size + chunk - 1) / chunk; }
 __device__ __forceinline__ bool whole_multi(const GrepWork& w, uint64_t nch) { return nch >= 2 && nch <= w.whole_chunks; }
-__global__ void __launch_bounds__(32) k_grep_open(const gfs_ctx* c, const __grid_constant__ GrepWork w, const char* dir, uint32_t dir_len,
+__global__ void __launch_bounds__(32) k_grep_open(const __grid_constant__ gfs_ctx cv_, const __grid_constant__ GrepWork w, const char* dir, uint32_t dir_len,
                                                   uint32_t max_files) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   __shared__ __align__(16) char pbuf[kMaxPath + 32];
   __shared__ uint32_t f_s;
   const int lane = threadIdx.x;
@@ -898,9 +902,10 @@ __device__ __forceinline__ uint32_t item_chunks(const ItemDesc& d) { return ((d.
 // block scans chunk after chunk, counting in shared memory across chunks.
 // Thread 0 claims the next item and loads its descriptor while the block
 // works on the current one (the claim and the descriptor load are off the path).
-__global__ void __launch_bounds__(256, 3) k_grep_scan(const gfs_ctx* c, const __grid_constant__ GrepWork w, uint32_t chunk, uint64_t* hits,
+__global__ void __launch_bounds__(256, 3) k_grep_scan(const __grid_constant__ gfs_ctx cv_, const __grid_constant__ GrepWork w, uint32_t chunk, uint64_t* hits,
                                                    uint64_t hit_cap, uint64_t* totals, uint32_t* rec,
                                                    uint64_t rec_cap) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) uint8_t sm[];
   const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31, wid = tid >> 5;
   const uint32_t buf_bytes = (kPre + chunk + kHalo + kSlack + 15) & ~15u;
@@ -1279,9 +1284,10 @@ struct WPageWin {
   }
 };
 
-__global__ void __launch_bounds__(256) k_grep_wscan(const gfs_ctx* c, const __grid_constant__ GrepWork w,
+__global__ void __launch_bounds__(256) k_grep_wscan(const __grid_constant__ gfs_ctx cv_, const __grid_constant__ GrepWork w,
                                                     uint64_t* hits, uint64_t hit_cap, uint64_t* totals,
                                                     uint32_t* rec, uint64_t rec_cap) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) uint8_t sm[];
   const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
   const uint32_t slots = w.cslots, tmask = slots - 1;
@@ -1444,7 +1450,8 @@ __global__ void __launch_bounds__(256) k_grep_wscan(const gfs_ctx* c, const __gr
   }
 }
 
-__global__ void k_grep_close(const gfs_ctx* c, const __grid_constant__ GrepWork w) {
+__global__ void k_grep_close(const __grid_constant__ gfs_ctx cv_, const __grid_constant__ GrepWork w) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const uint32_t nfiles = (uint32_t)w.vars[V_NFILES];
   for (uint32_t f = blockIdx.x; f < nfiles; f += gridDim.x) {
     const int fd = w.fd[f];
@@ -1733,7 +1740,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   const char* d_list = as.str(1);
   const char* d_dir = as.str(2);
 
-  const gfs_ctx* c = gfs_device_ctx(h);
+  const gfs_ctx c = gfs_launch::ctx_val(h);
   static unsigned long long* d_prof = nullptr;  // GFS_GREP_PROF=1 (diagnostics only)
   w.prof = nullptr;
   if (getenv("GFS_GREP_PROF") && *getenv("GFS_GREP_PROF") == '1') {

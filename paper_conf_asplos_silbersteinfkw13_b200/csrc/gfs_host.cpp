@@ -1144,6 +1144,7 @@ extern "C" void gfs_internal_args_done(gfs_handle* h, int slot, cudaStream_t s) 
 }
 
 extern "C" int gfs_internal_device(gfs_handle* h) { return h ? h->cfg.device : -1; }
+extern "C" const gfs_ctx* gfs_internal_host_ctx(gfs_handle* h) { return h ? &h->h : nullptr; }
 
 // ------------------------------------------------------------------ peer caches (NEXT-1)
 namespace {

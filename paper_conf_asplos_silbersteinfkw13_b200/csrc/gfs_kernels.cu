@@ -93,9 +93,10 @@ __device__ __forceinline__ void note_err(int64_t* d_err, int64_t r) {
   if (r < 0 && d_err) atomicMin((long long*)d_err, (long long)r);
 }
 
-__global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint32_t ncalls, const uint64_t* off,
+__global__ void k_gread_calls(const __grid_constant__ gfs_ctx cv_, const char* path, int mode, uint32_t ncalls, const uint64_t* off,
                               const uint64_t* len, const uint64_t* dstoff, uint8_t* dst, int64_t* ret,
                               uint32_t smem_bytes) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) uint8_t smem[];
   const int tid = threadIdx.x;
   const int fd = gopen(c, path, mode >> 8);  // open flags ride in the high bits (O_RDONLY or O_RDWR)
@@ -140,9 +141,10 @@ __global__ void k_gread_calls(const gfs_ctx* c, const char* path, int mode, uint
 // gclose_warp): warp w of the grid issues calls w, w + nwarps, ...
 // mode 4: into global memory; mode 5: into the warp's shared buffer
 // (smem_bytes per warp) at off % 16, then copied out.
-__global__ void k_gread_calls_warp(const gfs_ctx* c, const char* path, int mode, uint32_t ncalls,
+__global__ void k_gread_calls_warp(const __grid_constant__ gfs_ctx cv_, const char* path, int mode, uint32_t ncalls,
                                    const uint64_t* off, const uint64_t* len, const uint64_t* dstoff, uint8_t* dst,
                                    int64_t* ret, uint32_t smem_bytes) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) uint8_t smem[];
   const int lane = threadIdx.x & 31, wib = threadIdx.x >> 5;
   const uint32_t gw = blockIdx.x * (blockDim.x >> 5) + wib, nw = gridDim.x * (blockDim.x >> 5);
@@ -169,8 +171,9 @@ __global__ void k_gread_calls_warp(const gfs_ctx* c, const char* path, int mode,
   if (fd >= 0) gclose_warp(c, fd);
 }
 
-__global__ void __launch_bounds__(256, 4) k_seqread(const gfs_ctx* c, const char* path, uint64_t file_off, uint64_t total, uint64_t chunk,
+__global__ void __launch_bounds__(256, 4) k_seqread(const __grid_constant__ gfs_ctx cv_, const char* path, uint64_t file_off, uint64_t total, uint64_t chunk,
                           int use_mmap, uint8_t* scratch, uint64_t* sum, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int tid = threadIdx.x, nthr = blockDim.x;
   const int fd = gopen(c, path, GFS_O_RDONLY);
   if (fd < 0) {
@@ -221,8 +224,10 @@ __global__ void __launch_bounds__(256, 4) k_seqread(const gfs_ctx* c, const char
 }
 
 template <bool kHint>
-__global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const char* path, int raw, const uint8_t* rawp, uint32_t chunk,
-                           uint32_t calls, const uint64_t* offs, uint64_t* sum, int64_t* err) {
+__global__ void __launch_bounds__(256, 4) k_randread(const __grid_constant__ gfs_ctx cv, const char* path, int raw,
+                                                     const uint8_t* rawp, uint32_t chunk, uint32_t calls,
+                                                     const uint64_t* offs, uint64_t* sum, int64_t* err) {
+  const gfs_ctx* c = &cv;  // the context by value: its fields come from the constant bank
   extern __shared__ __align__(16) uint8_t smem[];
   const int tid = threadIdx.x, nthr = blockDim.x;
   int fd = 0;
@@ -278,9 +283,10 @@ __global__ void __launch_bounds__(256, 4) k_randread(const gfs_ctx* c, const cha
 // memory (warp w takes calls w, w + nwarps, ...), so one warp's lookup never
 // stalls the block's other warps at a barrier. raw: the same per-warp TMA
 // copies without GPUfs.
-__global__ void __launch_bounds__(256) k_randread_warp(const gfs_ctx* c, const char* path, int raw,
+__global__ void __launch_bounds__(256) k_randread_warp(const __grid_constant__ gfs_ctx cv_, const char* path, int raw,
                                                        const uint8_t* rawp, uint32_t chunk, uint32_t calls,
                                                        const uint64_t* offs, uint64_t* sum, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) uint8_t smem[];
   __shared__ uint64_t raw_mbar[GFS_WARP_API_MAX_WARPS];
   const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5, nw = blockDim.x >> 5;
@@ -331,10 +337,11 @@ __global__ void __launch_bounds__(256) k_randread_warp(const gfs_ctx* c, const c
 // into one half of a double buffer while the whole block checksums the other
 // half, so a call's page-table walk and copy overlap the previous calls'
 // consumption. raw: the same schedule with plain TMA copies of d_raw.
-__global__ void __launch_bounds__(256) k_randread_async(const gfs_ctx* c, const char* path, int raw,
+__global__ void __launch_bounds__(256) k_randread_async(const __grid_constant__ gfs_ctx cv_, const char* path, int raw,
                                                         const uint8_t* rawp, uint32_t chunk, uint32_t calls,
                                                         uint32_t depth, const uint64_t* offs, uint64_t* sum,
                                                         int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) uint8_t smem[];
   __shared__ uint64_t raw_mbar;
   const int tid = threadIdx.x, nthr = blockDim.x, lane = tid & 31, wid = tid >> 5;
@@ -394,9 +401,10 @@ __global__ void __launch_bounds__(256) k_randread_async(const gfs_ctx* c, const 
   if (!raw) gclose(c, fd);
 }
 
-__global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
+__global__ void k_gwrite_calls(const __grid_constant__ gfs_ctx cv_, const char* path, uint32_t ncalls, const uint64_t* off,
                                const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret,
                                int flags) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, path, flags);
   for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
     int64_t r = fd < 0 ? fd : gwrite(c, fd, off[i], len[i], src + srcoff[i]);
@@ -409,9 +417,10 @@ __global__ void k_gwrite_calls(const gfs_ctx* c, const char* path, uint32_t ncal
 // [off[i], off[i] + len[i]) with GFS_PROT_WRITE, stores src bytes through the
 // pointer, optionally gmsync()s the page, and gmunmap()s. ret[i] = bytes
 // mapped (the prefix) or -errno.
-__global__ void k_mmap_write(const gfs_ctx* c, const char* path, uint32_t ncalls, const uint64_t* off,
+__global__ void k_mmap_write(const __grid_constant__ gfs_ctx cv_, const char* path, uint32_t ncalls, const uint64_t* off,
                              const uint64_t* len, const uint64_t* srcoff, const uint8_t* src, int64_t* ret,
                              int do_msync) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, path, GFS_O_RDWR);
   for (uint32_t i = blockIdx.x; i < ncalls; i += gridDim.x) {
     int64_t r = fd;
@@ -439,8 +448,9 @@ __global__ void k_mmap_write(const gfs_ctx* c, const char* path, uint32_t ncalls
 
 // C5 write side: every block gopen()s the (pinned, O_GWRONCE) file, gwrite()s
 // its contiguous share of [0, total) from `src` in `chunk`-byte calls, gclose()s.
-__global__ void k_seqwrite(const gfs_ctx* c, const char* path, uint64_t total, uint64_t chunk, const uint8_t* src,
+__global__ void k_seqwrite(const __grid_constant__ gfs_ctx cv_, const char* path, uint64_t total, uint64_t chunk, const uint8_t* src,
                            int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, path, GFS_O_GWRONCE);
   if (fd < 0) {
     if (threadIdx.x == 0) note_err(err, fd);
@@ -464,7 +474,8 @@ __global__ void k_seqwrite(const gfs_ctx* c, const char* path, uint64_t total, u
 // concurrent callers split the write-back between them (each waits for its own).
 // allow_busy: -EBUSY (a page claimed by a concurrent gfsync of this grid) is
 // not an error here; a strict single-block pass follows and catches the rest.
-__global__ void k_fsync_from_pin(const gfs_ctx* c, const int64_t* pinned_fd, int64_t* err, int allow_busy) {
+__global__ void k_fsync_from_pin(const __grid_constant__ gfs_ctx cv_, const int64_t* pinned_fd, int64_t* err, int allow_busy) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int64_t fd = *pinned_fd;
   if (fd < 0) {
     if (threadIdx.x == 0 && blockIdx.x == 0) note_err(err, fd);
@@ -474,14 +485,16 @@ __global__ void k_fsync_from_pin(const gfs_ctx* c, const int64_t* pinned_fd, int
   if (threadIdx.x == 0 && r < 0 && !(allow_busy && r == -EBUSY)) note_err(err, r);
 }
 
-__global__ void k_unpin(const gfs_ctx* c, const int64_t* pinned_fd, int64_t* err) {
+__global__ void k_unpin(const __grid_constant__ gfs_ctx cv_, const int64_t* pinned_fd, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int64_t fd = *pinned_fd;
   if (fd < 0) return;
   const int r = gclose(c, (int)fd);
   if (threadIdx.x == 0 && r < 0) note_err(err, r);
 }
 
-__global__ void k_fileop(const gfs_ctx* c, const char* path, int flags, int op, uint64_t arg, int64_t* ret) {
+__global__ void k_fileop(const __grid_constant__ gfs_ctx cv_, const char* path, int flags, int op, uint64_t arg, int64_t* ret) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   if (op == 6) {  // gfsync from every block of the grid (the pages split by claim), then a strict pass
     const int fd = gopen(c, path, flags);
     int r = fd;
@@ -539,13 +552,13 @@ GFS_API int gfs_run_gread(gfs_handle* h, void* stream, const char* path, int mod
     if (dyn > 200 * 1024) return -EINVAL;
     if (dyn > 48 * 1024)
       cudaFuncSetAttribute(k_gread_calls_warp, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)dyn);
-    k_gread_calls_warp<<<grid, block, dyn, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len, d_dstoff, d_dst,
+    k_gread_calls_warp<<<grid, block, dyn, s>>>(gfs_launch::ctx_val(h), dp, mode, ncalls, d_off, d_len, d_dstoff, d_dst,
                                                 d_ret, smem_bytes);
     return launch_err(cudaGetLastError());
   }
   if ((mode & 0xFF) >= 2 && smem_bytes > 48 * 1024)
     cudaFuncSetAttribute(k_gread_calls, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem_bytes);
-  k_gread_calls<<<grid, block, (mode & 0xFF) >= 2 ? smem_bytes : 0, s>>>(gfs_device_ctx(h), dp, mode, ncalls, d_off, d_len,
+  k_gread_calls<<<grid, block, (mode & 0xFF) >= 2 ? smem_bytes : 0, s>>>(gfs_launch::ctx_val(h), dp, mode, ncalls, d_off, d_len,
                                                                 d_dstoff, d_dst, d_ret, smem_bytes);
   return launch_err(cudaGetLastError());
 }
@@ -558,7 +571,7 @@ GFS_API int gfs_run_seqread(gfs_handle* h, void* stream, const char* path, uint6
   gfs_launch::ArgStage as(h, s);
   if (const int e = as.stage(&path, 1)) return e;
   const char* dp = as.str(0);
-  k_seqread<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, file_off, total, chunk, use_mmap, d_scratch, d_sum, d_err);
+  k_seqread<<<grid, block, 0, s>>>(gfs_launch::ctx_val(h), dp, file_off, total, chunk, use_mmap, d_scratch, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
 
@@ -575,8 +588,9 @@ GFS_API int gfs_run_randread(gfs_handle* h, void* stream, const char* path, int 
   const char* dp = raw == 1 ? nullptr : as.str(0);
   auto kern = raw == 2 ? k_randread<true> : k_randread<false>;
   if (chunk > 48 * 1024) cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)chunk);
-  kern<<<grid, block, chunk, s>>>(raw == 1 ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk, calls_per_block,
-                                  d_off, d_sum, d_err);
+  gfs_ctx cv{};
+  if (raw != 1) cv = *gfs_internal_host_ctx(h);
+  kern<<<grid, block, chunk, s>>>(cv, dp, raw, d_raw, chunk, calls_per_block, d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
 
@@ -593,7 +607,7 @@ GFS_API int gfs_run_randread_warp(gfs_handle* h, void* stream, const char* path,
   const char* dp = raw ? nullptr : as.str(0);
   const uint32_t smem = chunk * (block / 32);
   if (smem > 48 * 1024) cudaFuncSetAttribute(k_randread_warp, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-  k_randread_warp<<<grid, block, smem, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk,
+  k_randread_warp<<<grid, block, smem, s>>>(gfs_launch::ctx_val(raw ? nullptr : h), dp, raw, d_raw, chunk,
                                              calls_per_block, d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
@@ -611,7 +625,7 @@ GFS_API int gfs_run_randread_async(gfs_handle* h, void* stream, const char* path
   const char* dp = raw ? nullptr : as.str(0);
   const uint32_t smem = chunk * depth * 2;
   if (smem > 48 * 1024) cudaFuncSetAttribute(k_randread_async, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-  k_randread_async<<<grid, block, smem, s>>>(raw ? nullptr : gfs_device_ctx(h), dp, raw, d_raw, chunk,
+  k_randread_async<<<grid, block, smem, s>>>(gfs_launch::ctx_val(raw ? nullptr : h), dp, raw, d_raw, chunk,
                                               calls_per_block, depth, d_off, d_sum, d_err);
   return launch_err(cudaGetLastError());
 }
@@ -625,7 +639,7 @@ GFS_API int gfs_run_gwrite(gfs_handle* h, void* stream, const char* path, uint32
   gfs_launch::ArgStage as(h, s);
   if (const int e = as.stage(&path, 1)) return e;
   const char* dp = as.str(0);
-  k_gwrite_calls<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, flags);
+  k_gwrite_calls<<<grid, block, 0, s>>>(gfs_launch::ctx_val(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, flags);
   return launch_err(cudaGetLastError());
 }
 
@@ -637,7 +651,7 @@ GFS_API int gfs_run_mmap_write(gfs_handle* h, void* stream, const char* path, ui
   gfs_launch::ArgStage as(h, s);
   if (const int e = as.stage(&path, 1)) return e;
   const char* dp = as.str(0);
-  k_mmap_write<<<grid, block, 0, s>>>(gfs_device_ctx(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, do_msync);
+  k_mmap_write<<<grid, block, 0, s>>>(gfs_launch::ctx_val(h), dp, ncalls, d_off, d_len, d_srcoff, d_src, d_ret, do_msync);
   return launch_err(cudaGetLastError());
 }
 
@@ -650,7 +664,7 @@ GFS_API int gfs_run_seqwrite(gfs_handle* h, void* stream, const char* path, uint
   gfs_launch::ArgStage as(h, s);
   if (const int e = as.stage(&path, 1)) return e;
   const char* dp = as.str(0);
-  const gfs_ctx* c = gfs_device_ctx(h);
+  const gfs_ctx c = gfs_launch::ctx_val(h);
   // pin: one open held across the launches, so the writers' gclose never
   // closes the file (a later O_GWRONCE open would start a new incarnation)
   k_fileop<<<1, 256, 0, s>>>(c, dp, GFS_O_GWRONCE, 4, 0, d_tmp);
@@ -671,11 +685,11 @@ GFS_API int gfs_run_fileop(gfs_handle* h, void* stream, const char* path, int fl
   if (op == 6) {  // parallel gfsync: arg = grid; *d_ret = 0 or the most negative error
     if (arg == 0 || arg > 65535) return -EINVAL;
     cudaMemsetAsync(d_ret, 0, 8, s);
-    k_fileop<<<(uint32_t)arg, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, 6, 0, d_ret);
-    k_fileop<<<1, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, 6, 1, d_ret);  // strict: every page clean now
+    k_fileop<<<(uint32_t)arg, 256, 0, s>>>(gfs_launch::ctx_val(h), dp, flags, 6, 0, d_ret);
+    k_fileop<<<1, 256, 0, s>>>(gfs_launch::ctx_val(h), dp, flags, 6, 1, d_ret);  // strict: every page clean now
     return launch_err(cudaGetLastError());
   }
-  k_fileop<<<1, 256, 0, s>>>(gfs_device_ctx(h), dp, flags, op, arg, d_ret);
+  k_fileop<<<1, 256, 0, s>>>(gfs_launch::ctx_val(h), dp, flags, op, arg, d_ret);
   return launch_err(cudaGetLastError());
 }
 

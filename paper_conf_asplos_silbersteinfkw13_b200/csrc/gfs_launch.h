@@ -11,8 +11,21 @@
 extern "C" int gfs_internal_args(gfs_handle* h, cudaStream_t s, const char* const* strs, int n, char** d_out);
 extern "C" void gfs_internal_args_done(gfs_handle* h, int slot, cudaStream_t s);
 extern "C" int gfs_internal_device(gfs_handle* h);
+// The host copy of the handle's context (what gfs_device_ctx points to on the
+// device, kept in step with it): launchers pass it BY VALUE as a
+// __grid_constant__ kernel parameter, so the kernel reads the context's
+// fields from the constant bank instead of L1/L2.
+extern "C" const gfs_ctx* gfs_internal_host_ctx(gfs_handle* h);
 
 namespace gfs_launch {
+// The context a kernel takes by value (zeros for kernels launched without a
+// handle, e.g. the raw baselines, which never read it).
+inline gfs_ctx ctx_val(gfs_handle* h) {
+  gfs_ctx v{};
+  if (const gfs_ctx* p = h ? gfs_internal_host_ctx(h) : nullptr) v = *p;
+  return v;
+}
+
 
 // Scope of one launcher call: makes the handle's device current, stages the
 // strings in a slot of the handle's ring, and — when the launcher returns,

@@ -36,7 +36,8 @@ __device__ __forceinline__ void mv_err(int64_t* err, int64_t r) {
   if (r < 0 && err) atomicMin((long long*)err, (long long)r);
 }
 
-__global__ void k_mv_trunc(const gfs_ctx* c, const char* y_path, int64_t* err) {
+__global__ void k_mv_trunc(const __grid_constant__ gfs_ctx cv_, const char* y_path, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, y_path, GFS_O_GWRONCE);
   if (fd < 0) {
     if (threadIdx.x == 0) mv_err(err, fd);
@@ -49,7 +50,8 @@ __global__ void k_mv_trunc(const gfs_ctx* c, const char* y_path, int64_t* err) {
   // a new incarnation)
 }
 
-__global__ void k_mv_x(const gfs_ctx* c, const char* x_path, uint64_t cols, float* x, int64_t* err) {
+__global__ void k_mv_x(const __grid_constant__ gfs_ctx cv_, const char* x_path, uint64_t cols, float* x, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, x_path, GFS_O_RDONLY);
   if (fd < 0) {
     if (threadIdx.x == 0 && blockIdx.x == 0) mv_err(err, fd);
@@ -77,9 +79,10 @@ __device__ __forceinline__ double block_sum(double v, double* red) {
 }
 
 // Rows [row0, row0 + nrows) of A; y (file and d_y) holds those rows only.
-__global__ void __launch_bounds__(256) k_mv_rows(const gfs_ctx* c, const char* a_path, const char* y_path,
+__global__ void __launch_bounds__(256) k_mv_rows(const __grid_constant__ gfs_ctx cv_, const char* a_path, const char* y_path,
                                                   uint64_t row0, uint64_t nrows, uint64_t cols, const float* x,
                                                   float* y_dev, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) float ys[];  // this block's y slice
   __shared__ double red[32];
   const int tid = threadIdx.x, nthr = blockDim.x;
@@ -141,7 +144,8 @@ __global__ void __launch_bounds__(256) k_mv_rows(const gfs_ctx* c, const char* a
   gclose(c, fy);
 }
 
-__global__ void k_mv_sync(const gfs_ctx* c, const char* y_path, int64_t* err) {
+__global__ void k_mv_sync(const __grid_constant__ gfs_ctx cv_, const char* y_path, int64_t* err) {
+  const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   const int fd = gopen(c, y_path, GFS_O_GWRONCE);
   if (fd < 0) {
     if (threadIdx.x == 0) mv_err(err, fd);
@@ -167,7 +171,7 @@ GFS_API int gfs_matvec_rows(gfs_handle* h, void* stream, const char* a_path, con
   gfs_launch::ArgStage as(h, s);
   const char* ps[3] = {a_path, x_path, y_path};
   if (const int e = as.stage(ps, 3)) return e;
-  const gfs_ctx* c = gfs_device_ctx(h);
+  const gfs_ctx c = gfs_launch::ctx_val(h);
   const char* da = as.str(0);
   const char* dx = as.str(1);
   const char* dy = as.str(2);
