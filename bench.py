@@ -42,6 +42,10 @@ import time
 
 import numpy as np
 
+# Load every kernel when the CUDA context is created (not at its first launch):
+# a "cold" grep or fill then measures the cache, not lazy module loading.
+os.environ.setdefault("CUDA_MODULE_LOADING", "EAGER")
+
 ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
 

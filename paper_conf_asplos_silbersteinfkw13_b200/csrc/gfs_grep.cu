@@ -105,6 +105,7 @@ struct GrepWork {
   // (file, word) -> count table
   uint64_t* pair;         // slot i: pair[2i] = (file << 32) | word (or empty), pair[2i+1] = count
   uint64_t pair_mask;
+  uint32_t* ptouch;       // one bit per 256 slots that hold (or held) a pair this run: compact skips the rest
   // output records, staged in pages: a block reserves a page of kRecPage
   // records with ONE atomic and fills it privately (a global counter bumped
   // per record or per warp serialises at one L2 address, ~14 ns each);
@@ -289,6 +290,8 @@ __global__ void k_grep_init(const __grid_constant__ GrepWork w, uint32_t max_wor
   if (t < V_NVARS) w.vars[t] = 0;
 }
 
+__host__ __device__ __forceinline__ uint64_t ptouch_words(uint64_t slots) { return (slots / 256 + 31) / 32; }
+
 // The (file, word) table is emptied by every successful run's compact; only
 // a fresh work buffer or a failed run leaves it dirty.
 __global__ void k_grep_pairclear(const __grid_constant__ GrepWork w) {
@@ -298,6 +301,8 @@ __global__ void k_grep_pairclear(const __grid_constant__ GrepWork w) {
     w.pair[2 * i] = kPairEmpty;
     w.pair[2 * i + 1] = 0;
   }
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < ptouch_words(w.pair_mask + 1); i += stride)
+    w.ptouch[i] = 0;
 }
 
 // --------------------------------------------------------------- dictionary
@@ -685,6 +690,11 @@ __device__ __noinline__ void pair_add(const GrepWork& w, uint32_t f, uint32_t k,
                                              (unsigned long long)key);
     if (cur == kPairEmpty || cur == key) {
       atomicAdd((unsigned long long*)&w.pair[2 * slot + 1], (unsigned long long)cnt);
+      if (cur == kPairEmpty) {  // a new pair: its 256-slot region is one compact must visit
+        const uint64_t r = slot >> 8;
+        const uint32_t bit = 1u << (r & 31);
+        if (!(*(volatile uint32_t*)&w.ptouch[r >> 5] & bit)) atomicOr(&w.ptouch[r >> 5], bit);
+      }
       return;
     }
   }
@@ -1476,13 +1486,18 @@ __global__ void __launch_bounds__(256) k_grep_compact(const __grid_constant__ Gr
   const uint64_t n = w.pair_mask + 1;  // a power of two >= 1024
   constexpr int kPer = 8;                // slots per thread (128 bytes in flight per thread)
   for (uint64_t blk = blockIdx.x; blk * 256 * kPer < n; blk += gridDim.x) {
+    // the 8 regions of 256 slots this block covers (one per warp): only the
+    // ones a pair was inserted into this run are read
+    const uint32_t tb = (w.ptouch[blk >> 2] >> ((blk & 3) * 8)) & 0xFFu;
+    if (!tb) continue;  // (the same for every thread of the block)
+    const bool mine = (tb >> wid) & 1u;
     const uint64_t i0 = blk * 256 * kPer + (uint64_t)tid * kPer;
     uint4* src = (uint4*)(w.pair + 2 * i0);
     uint64_t key[kPer], cnt[kPer];
     uint32_t nv = 0;
 #pragma unroll
     for (int q = 0; q < kPer; ++q) {
-      const uint4 v = i0 < n ? src[q] : make_uint4(0xFFFFFFFFu, 0xFFFFFFFFu, 0u, 0u);  // (n >= 1024: whole groups)
+      const uint4 v = (mine && i0 < n) ? src[q] : make_uint4(0xFFFFFFFFu, 0xFFFFFFFFu, 0u, 0u);  // (n >= 1024: whole groups)
       key[q] = ((uint64_t)v.y << 32) | v.x;
       cnt[q] = ((uint64_t)v.w << 32) | v.z;
       nv += key[q] != kPairEmpty;
@@ -1517,6 +1532,7 @@ __global__ void __launch_bounds__(256) k_grep_compact(const __grid_constant__ Gr
       ++idx;
       src[q] = make_uint4(0xFFFFFFFFu, 0xFFFFFFFFu, 0u, 0u);  // empty again for the next run
     }
+    if (tid == 0) atomicAnd(&w.ptouch[blk >> 2], ~(0xFFu << ((blk & 3) * 8)));  // regions empty again
     __syncthreads();  // warp_tot / base_s reuse
   }
   if (tid == 0) rec_close(w, page_s, used_s);
@@ -1590,7 +1606,7 @@ uint64_t pow2_at_least(uint64_t x) {
 }
 
 struct Layout {
-  uint64_t off[18];
+  uint64_t off[19];
   uint64_t total;
   uint64_t max_items, tcap, pcap, max_pages;
   uint32_t flog2;
@@ -1627,9 +1643,10 @@ Layout layout(const gfs_grep_params* p) {
       V_NVARS * 8,                                         // 14 vars
       K_NKEEP * 8,                                         // 15 keep (persistent)
       (1ull << L.flog2) / 8,                               // 16 word filter
+      ptouch_words(L.pcap) * 4,                            // 17 touched regions of the pair table
   };
   uint64_t o = 0;
-  for (int i = 0; i < 17; ++i) {
+  for (int i = 0; i < 18; ++i) {
     L.off[i] = o;
     o += (sizes[i] + 255) & ~255ull;
   }
@@ -1717,6 +1734,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   }
   w.pair = (uint64_t*)(base + L.off[10]);
   w.pair_mask = L.pcap - 1;
+  w.ptouch = (uint32_t*)(base + L.off[17]);
   w.rpool = (uint32_t*)(base + L.off[11]);
   w.page_used = (uint32_t*)(base + L.off[12]);
   w.page_base = (uint64_t*)(base + L.off[13]);
