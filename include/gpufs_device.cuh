@@ -216,6 +216,17 @@ constexpr uint64_t kRefDec = ~0ull;  // ref - 1 (never borrows: the ref being dr
 __device__ __forceinline__ uint64_t fl64(uint32_t flags) { return ~(uint64_t)flags; }  // and-mask clearing flags
 // Leaf slot value for frame f of generation gen.
 __device__ __forceinline__ uint64_t slot_val(uint32_t f, uint32_t gen) { return ((uint64_t)gen << 32) | (f + 1u); }
+// Bit 31 of a leaf slot's low word: the slot was installed and no lookup has yet
+// seen its frame's fill complete. Installs write slot_val_fill(); the first
+// lookup that validates the frame (same generation, no FILLING) clears it.
+// A slot without the bit therefore names an incarnation whose bytes were
+// complete before the slot was read (FILLING is set once per generation, at
+// install, and cleared once): gread's one-page fast path may start its copy
+// from such a frame before its reference is confirmed (the reference then
+// decides whether the copy is kept, gread_t).
+constexpr uint32_t kSlotFill = 0x80000000u;
+__device__ __forceinline__ uint64_t slot_val_fill(uint32_t f, uint32_t gen) { return slot_val(f, gen) | kSlotFill; }
+__device__ __forceinline__ uint32_t slot_frame(uint64_t s) { return ((uint32_t)s & ~kSlotFill) - 1u; }
 // Claim frame f for exclusive use (EVICTING) if its low word is exactly `low`
 // (0: unreferenced, no flags). Keeps the generation.
 __device__ __forceinline__ bool claim_frame(uint64_t* st, uint32_t low) {
@@ -978,8 +989,10 @@ __device__ __forceinline__ void frame_abandon(const gfs_ctx* c, uint32_t f) {
 // caller's block holds the file open. All accesses are strong gpu-scope
 // operations served at L2, so no L1 line can be stale. Returns the frame, or
 // -1 to take the full (acquire/release) path.
-__device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs, uint64_t page,
-                                           uint64_t* leaf_cache = nullptr) {
+// The leaf slot of `page` (relaxed walk, leaf cache), or nullptr when an
+// interior node is missing.
+__device__ __forceinline__ uint64_t* leaf_slot(const gfs_ctx* c, const FileSnap& fs, uint64_t page,
+                                               uint64_t* leaf_cache) {
   uint32_t node = fs.root;
   if (fs.height > 1) {
     const uint32_t key = (uint32_t)(page >> GFS_FANOUT_SHIFT);
@@ -990,16 +1003,24 @@ __device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs,
       for (int lvl = (int)fs.height - 1; lvl >= 1; --lvl) {
         node = (uint32_t)ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT +
                                   ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
-        if (!node) return -1;
+        if (!node) return nullptr;
       }
       if (leaf_cache) leaf_cache[key & (kLeafCache - 1)] = (((uint64_t)key + 1) << 32) | node;
     }
   }
-  const uint64_t s = ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
+  return c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u);
+}
+
+__device__ __forceinline__ int lookup_fast(const gfs_ctx* c, const FileSnap& fs, uint64_t page,
+                                           uint64_t* leaf_cache = nullptr) {
+  uint64_t* const sp = leaf_slot(c, fs, page, leaf_cache);
+  if (!sp) return -1;
+  const uint64_t s = ld_rlx64(sp);
   if (!(uint32_t)s) return -1;
-  const uint32_t f = (uint32_t)s - 1u;
+  const uint32_t f = slot_frame(s);
   const uint64_t old = a64_add_rlx(&c->f_state[f], 1ull);
   if ((old >> 32) == (s >> 32) && !((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
+    if ((uint32_t)s & kSlotFill) a64_cas(sp, s, s & ~(uint64_t)kSlotFill);  // the fill is complete: say so
     ctr(c, GFS_C_HIT);
     ctr(c, GFS_C_LOCKFREE);
     return (int)f;
@@ -1019,7 +1040,7 @@ __device__ __forceinline__ bool peek_busy(const gfs_ctx* c, const FileSnap& fs, 
   }
   const uint64_t s = ld_rlx64(c->nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
   if (!(uint32_t)s) return false;
-  const uint64_t st = ld_rlx64(&c->f_state[(uint32_t)s - 1u]);
+  const uint64_t st = ld_rlx64(&c->f_state[slot_frame(s)]);
   return (st >> 32) == (s >> 32) && ((uint32_t)st & (GFS_ST_FILLING | GFS_ST_EVICTING));
 }
 
@@ -1072,7 +1093,7 @@ __device__ __noinline__ int peer_take(const gfs_ctx* c, const FileSnap& fs, uint
                                       ((uint32_t)(page >> (GFS_FANOUT_SHIFT * lvl)) & 255u));
       if (!node || node >= P.max_nodes) break;  // type-stable nodes: a racing free reads as a miss
       const uint64_t sl = ld_rlx_sys64(P.nodes + (size_t)node * GFS_FANOUT + ((uint32_t)page & 255u));
-      const uint32_t f = (uint32_t)sl - 1u;
+      const uint32_t f = slot_frame(sl);
       if (!(uint32_t)sl || f >= P.nframes) break;
       const uint64_t old = a64_add_sys(&P.f_state[f], 1ull);
       fence_sys();  // the checks and the copy below read after the reference is held
@@ -1155,7 +1176,7 @@ __device__ __noinline__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint
     const uint64_t s = ld_acq64(slot);
     bool done = false;
     if ((uint32_t)s) {
-      const uint32_t f = (uint32_t)s - 1u;
+      const uint32_t f = slot_frame(s);
       const uint64_t old = a64_add_acq(&c->f_state[f], 1ull);
       // same generation as the slot <=> the frame still holds this page (the
       // tag check is kept as a belt-and-braces test on the slow path)
@@ -1241,7 +1262,7 @@ __device__ __noinline__ Lk lookup_try(const gfs_ctx* c, const FileSnap& fs, uint
       out.frame = g;
       break;
     }
-    const bool won = a64_cas(slot, s, slot_val((uint32_t)g, gen)) == s;
+    const bool won = a64_cas(slot, s, slot_val_fill((uint32_t)g, gen)) == s;
     if (!won) {
       if (st != -1) fill_src_free(c, st);
       frame_abandon(c, (uint32_t)g);
@@ -1426,7 +1447,7 @@ __device__ __noinline__ int ra_issue(const gfs_ctx* c, const FileSnap& fs, uint6
   }
   const uint64_t s = ld_acq64(slot);
   if ((uint32_t)s) {  // only a stale slot (frame reassigned, or failed and not refilling) is replaced
-    const uint64_t fst = ld_acq64(&c->f_state[(uint32_t)s - 1u]);
+    const uint64_t fst = ld_acq64(&c->f_state[slot_frame(s)]);
     const bool stale = (fst >> 32) != (s >> 32) ||
                        (((uint32_t)fst & GFS_ST_ERROR) && !((uint32_t)fst & GFS_ST_FILLING));
     if (!stale) {
@@ -1441,7 +1462,7 @@ __device__ __noinline__ int ra_issue(const gfs_ctx* c, const FileSnap& fs, uint6
     return -1;
   }
   st_rel64(&c->f_pf[g], GFS_PF_POSTING);  // lookups that find it now wait (busy) instead of adopting
-  if (a64_cas(slot, s, slot_val((uint32_t)g, gen)) != s) {
+  if (a64_cas(slot, s, slot_val_fill((uint32_t)g, gen)) != s) {
     st_rlx64(&c->f_pf[g], 0);
     frame_abandon(c, (uint32_t)g);
     stage_free(c, st);
@@ -1748,7 +1769,7 @@ __device__ int claim_dirty(const gfs_ctx* c, const FileSnap& fs, uint64_t p) {
   if (!slot) return -1;
   const uint64_t s = ld_acq64(slot);
   if (!(uint32_t)s) return -1;
-  const uint32_t f = (uint32_t)s - 1u;
+  const uint32_t f = slot_frame(s);
   const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
   if (ld_acq64(&c->f_tag[f]) != want || ld_rlx(&c->f_lo[f]) == GFS_DIRTY_NONE) return -1;
   if (!claim_frame(&c->f_state[f], 0u))
@@ -1787,7 +1808,7 @@ __device__ int drop_pages(const gfs_ctx* c, const FileSnap& fs, uint64_t pb, uin
     if (!slot) continue;
     const uint64_t s = ld_acq64(slot);
     if (!(uint32_t)s) continue;
-    const uint32_t f = (uint32_t)s - 1u;
+    const uint32_t f = slot_frame(s);
     const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)p;
     if (ld_acq64(&c->f_tag[f]) != want) continue;
     if (!claim_frame(&c->f_state[f], 0u)) {
@@ -1927,7 +1948,7 @@ __device__ int open_leader(const gfs_ctx* c, const char* path, uint32_t n, uint6
           uint32_t gen = 0;
           const int g = alloc_frame(c, (uint64_t)e->uid << 32, i, &gen);
           if (g >= 0) {
-            if (a64_cas(slot, 0ull, slot_val((uint32_t)g, gen)) == 0ull) {
+            if (a64_cas(slot, 0ull, detail::slot_val_fill((uint32_t)g, gen)) == 0ull) {
               pf->frame = g;
               pf->stage = pst;
               pf->nbytes = nb;
@@ -2281,8 +2302,42 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
       const uint32_t cnt = (uint32_t)((q1 - q0 + 1) < B ? (q1 - q0 + 1) : B);
       if (tid < (int)cnt) {
         const FileSnap fs0 = sc.fs;
-        int f = hinted >= 0 ? hinted : fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
-        if (f < 0) {
+        const bool quick_ok =
+            q0 == q1 && n0 < (1 << 20) && __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0;
+        if (fast && hinted < 0 && quick_ok && !(c->flags & GFS_F_NO_SPECULATE)) {
+          // Speculative one-page hit (lane 0; cnt == 1): a slot whose fill is known
+          // complete (no kSlotFill) lets the copy start with the reference still in
+          // flight. The reference's old state decides: same generation and no
+          // FILLING / EVICTING / ERROR means the frame held this page's bytes from
+          // the slot read on (a generation is never reused), so the copy is kept;
+          // otherwise the reference is dropped, the copy waited out (it may not
+          // land after dst is reused) and the call takes the normal path.
+          uint64_t* const sp = leaf_slot(c, fs0, q0, sc.lc_ok ? sc.leaf : nullptr);
+          const uint64_t sv = sp ? ld_rlx64(sp) : 0ull;
+          if ((uint32_t)sv && !((uint32_t)sv & kSlotFill)) {
+            const uint32_t fs_ = slot_frame(sv);
+            const uint64_t old = a64_add_rlx(&c->f_state[fs_], 1ull);
+            asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // prior generic use of dst
+            uint64_t* mb = &sc.mbar;
+            const uint8_t* src = frame_ptr(c, fs_) + (off & (P - 1));
+            mbar_expect_tx(mb, span_mid(src, (uint32_t)n0));
+            tma_span((uint8_t*)dst, src, (uint32_t)n0, mb);
+            if ((old >> 32) == (sv >> 32) && !((uint32_t)old & (GFS_ST_FILLING | GFS_ST_EVICTING | GFS_ST_ERROR))) {
+              ctr(c, GFS_C_HIT);
+              ctr(c, GFS_C_LOCKFREE);
+              sc.frame[0] = (int32_t)fs_;
+              quick = 1;
+            } else {
+              r64_add_rlx(&c->f_state[fs_], kRefDec);
+              mbar_wait(mb, sc.mbar_phase);
+              sc.mbar_phase ^= 1u;
+            }
+          }
+        }
+        int f = quick ? -2 : hinted >= 0 ? hinted : fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
+        if (quick) {
+          // the speculative copy is in flight (above)
+        } else if (f < 0) {
           const Lk r = lookup_try(c, fs0, q0 + tid);
           sc.frame[tid] = r.frame;
           sc.fill[tid] = r.fill;
@@ -2985,7 +3040,7 @@ __device__ inline int gftruncate(const gfs_ctx* c, int fd, uint64_t size) {
     uint64_t* slot = walk(c, fs.root, fs.height, b, false, nullptr);
     const uint64_t sv = slot ? ld_acq64(slot) : 0;
     if ((uint32_t)sv) {
-      const uint32_t f = (uint32_t)sv - 1u;
+      const uint32_t f = detail::slot_frame(sv);
       const uint64_t want = ((uint64_t)fs.uid << 32) | (uint32_t)b;
       if (ld_acq64(&c->f_tag[f]) == want) {
         if (!claim_frame(&c->f_state[f], 0u)) {

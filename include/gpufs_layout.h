@@ -39,6 +39,7 @@ extern "C" {
 #define GFS_F_LOCKED_TRAVERSAL 1u /* K5 ablation: every lookup takes the file lock */
 #define GFS_F_NO_DMA_COMPLETION 2u /* fallback: completion via memcpy instead of stream write-value */
 #define GFS_F_EXPORTED 4u          /* set by gfs_export: frames are published at system scope for peers */
+#define GFS_F_NO_SPECULATE 8u      /* ablation: gread's one-page hits wait for the reference before copying */
 
 /* ---- frame state word (pframe "state", 64 bits) -------------------------
  * bits 32..63 generation: +1 each time the frame is (re)assigned to a page.

@@ -30,7 +30,8 @@ def timed(fn, reps=5):
     return float(np.mean(ts))
 
 
-with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, daemon_threads=12) as fs:
+flags = int(os.environ.get("K4_FLAGS", "0"))  # 8: GFS_F_NO_SPECULATE (A/B of the speculative hit copy)
+with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, daemon_threads=12, flags=flags) as fs:
     assert fs.seqread(path, size, P, grid=296)[1] == 0
     raw = torch.empty(size, dtype=torch.uint8, device=dev)
     raw.copy_(torch.from_file(path, shared=False, size=size, dtype=torch.uint8))
@@ -52,5 +53,5 @@ with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, daemon_threads=12) as 
             r = fs.randread(path if kind == "gpufs" else None, chunk, d_off, grid, block=block,
                             raw=raw if kind == "raw" else None)
             res[kind] = (grid * calls * chunk / ms / 1e6, r == (want, 0))
-        print(f"block {block} x {per_sm}/SM: gpufs {res['gpufs'][0]:.0f} GB/s raw {res['raw'][0]:.0f} GB/s "
+        print(f"flags {flags} block {block} x {per_sm}/SM: gpufs {res['gpufs'][0]:.0f} GB/s raw {res['raw'][0]:.0f} GB/s "
               f"ratio {res['gpufs'][0] / res['raw'][0]:.3f} parity {res['gpufs'][1]} {res['raw'][1]}", flush=True)
