@@ -306,3 +306,28 @@ def test_randread_hint_checksum_and_no_leaked_references(g, shmdir):
             assert fs.randread(path, chunk, offs, grid, hint=True) == (expect, 0)
         s, err = fs.seqread(other, size, P, grid=24)
         assert err == 0 and s == oracle.checksum(other, 0, size)
+
+
+def test_speculative_hit_copy_under_churn(g, shmdir):
+    """gread's speculative one-page copy (the TMA starts before the reference is
+    confirmed, for slots whose fill is known complete): two files alternate
+    through a cache of 16 frames for 2 x 48 pages, so slots routinely name
+    frames that were evicted and refilled with another file's page (the
+    generation check must reject those copies); the checksums over every call
+    equal the oracle's, with speculation on and off (GFS_F_NO_SPECULATE), and the
+    counters show both accepted speculative hits and misses."""
+    P = 1 << 16
+    size = 48 * P
+    chunk = 16384
+    paths = [gen.splitmix_file(os.path.join(shmdir, f"spec{i}.bin"), size, seed=60 + i) for i in range(2)]
+    grid, calls = 12, 64
+    rng = np.random.default_rng(11)
+    offs = [(rng.integers(0, size // chunk, size=grid * calls) * chunk).astype(np.uint64) for _ in range(2)]
+    expect = [sum(oracle.checksum(p, int(o), chunk) for o in of) % (1 << 64) for p, of in zip(paths, offs)]
+    for flags in (0, 8):  # 8 = GFS_F_NO_SPECULATE
+        with g.GpuFS(cache_bytes=16 * P, page_size=P, timeout_ms=30000, daemon_threads=4, flags=flags) as fs:
+            for rep in range(4):
+                for i in (0, 1):
+                    assert fs.randread(paths[i], chunk, offs[i], grid, block=96) == (expect[i], 0), (flags, rep, i)
+            st = fs.stats()
+        assert st["miss"] > 0 and st["hit"] > 0 and st["evict"] > 0
