@@ -80,13 +80,12 @@ __device__ __forceinline__ double block_sum(double v, double* red) {
 
 // Rows [row0, row0 + nrows) of A; y (file and d_y) holds those rows only.
 __global__ void __launch_bounds__(256) k_mv_rows(const __grid_constant__ gfs_ctx cv_, const char* a_path, const char* y_path,
-                                                  uint64_t row0, uint64_t nrows, uint64_t cols, const float* x,
-                                                  float* y_dev, int64_t* err) {
+                                                  uint64_t row0, uint64_t nrows, uint64_t cols, uint64_t per,
+                                                  const float* x, float* y_dev, int64_t* err) {
   const gfs_ctx* c = &cv_;  // by value: the context's fields come from the constant bank
   extern __shared__ __align__(16) float ys[];  // this block's y slice
   __shared__ double red[32];
   const int tid = threadIdx.x, nthr = blockDim.x;
-  const uint64_t per = (nrows + gridDim.x - 1) / gridDim.x;
   const uint64_t r0 = row0 + blockIdx.x * per, r1 = r0 + per < row0 + nrows ? r0 + per : row0 + nrows;
   if (r0 >= r1) return;
   const int fa = gopen(c, a_path, GFS_O_RDONLY);
@@ -165,7 +164,18 @@ GFS_API int gfs_matvec_rows(gfs_handle* h, void* stream, const char* a_path, con
   if (!h || !a_path || !x_path || !y_path || !d_x || !d_err || rows == 0 || cols == 0 || grid == 0 ||
       block == 0 || block > 256 || (block & 31) || nrows == 0 || row0 >= rows || nrows > rows - row0)
     return -EINVAL;
-  const uint64_t per = (nrows + grid - 1) / grid;
+  // Rows per block: ceil(nrows / grid), rounded up to whole cache pages when a
+  // page holds whole rows, so no page is shared by two blocks (a shared page
+  // makes one block wait for the other's fill, or fetch it a second time after
+  // an eviction); blocks past the last row return at once.
+  uint64_t per = (nrows + grid - 1) / grid;
+  {
+    const uint64_t P = gfs_launch::ctx_val(h).page_size, rowb = cols * 4;
+    if (rowb <= P && P % rowb == 0 && (row0 * rowb) % P == 0) {
+      const uint64_t rpp = P / rowb;
+      per = (per + rpp - 1) / rpp * rpp;
+    }
+  }
   if (per * 4 > 160 * 1024) return -EINVAL;  // y slice must fit in shared memory: use more blocks
   cudaStream_t s = (cudaStream_t)stream;
   gfs_launch::ArgStage as(h, s);
@@ -180,7 +190,7 @@ GFS_API int gfs_matvec_rows(gfs_handle* h, void* stream, const char* a_path, con
   cudaMemsetAsync(d_err, 0, 8, s);
   k_mv_trunc<<<1, 128, 0, s>>>(c, dy, d_err);
   k_mv_x<<<64, 256, 0, s>>>(c, dx, cols, d_x, d_err);
-  k_mv_rows<<<grid, block, smem, s>>>(c, da, dy, row0, nrows, cols, d_x, d_y, d_err);
+  k_mv_rows<<<grid, block, smem, s>>>(c, da, dy, row0, nrows, cols, per, d_x, d_y, d_err);
   k_mv_sync<<<1, 256, 0, s>>>(c, dy, d_err);
   const cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) fprintf(stderr, "gfs_matvec: launch failed: %s\n", cudaGetErrorString(e));
