@@ -315,13 +315,14 @@ struct Scratch {
   uint32_t ra_f[16];
   uint64_t ra_v[16];
   // next-call hint (gread_hint): a page of the block's next gread, looked up
-  // and referenced while this call's copy was in flight; valid for hint_grid
-  // / hint_blk while hint_f >= 0, consumed or released by the next gread/gclose
+  // whose leaf slot was read while this call's copy was in flight (no
+  // reference is taken); valid for hint_grid / hint_blk while hint_ok
   uint64_t hint_grid;
   uint32_t hint_blk;
   int32_t hint_fd;
-  int32_t hint_f;
+  uint32_t hint_ok;
   uint64_t hint_page;
+  uint64_t hint_sv;
 };
 constexpr uint32_t kRA = 16;  // read-ahead fills a block tracks
 
@@ -2159,11 +2160,8 @@ __device__ inline int gclose_t(const gfs_ctx* c, int fd) {
   }
   if (G::tid() == 0) {
     if (sc.cached_fd == fd) sc.cached_fd = -1;
-    if constexpr (G::kBlock) {  // an unconsumed gread hint on this file
-      if (sc.hint_grid == detail::grid_id() && sc.hint_blk == G::key() && sc.hint_f >= 0 && sc.hint_fd == fd) {
-        detail::r64_add_rlx(&c->f_state[sc.hint_f], detail::kRefDec);
-        sc.hint_f = -1;
-      }
+    if constexpr (G::kBlock) {  // an unconsumed gread hint on this file (it holds nothing)
+      if (sc.hint_grid == detail::grid_id() && sc.hint_blk == G::key() && sc.hint_fd == fd) sc.hint_ok = 0;
     }
     sc.ret = detail::close_leader(c, fd);
   }
@@ -2288,13 +2286,13 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
     __syncwarp(nthr >= 32 ? 0xFFFFFFFFu : ((1u << nthr) - 1u));
     const int64_t n0 = sc.ret;
     uint32_t quick = 0;
-    // the previous call's hint: this call's first page, already referenced
-    int hinted = -1;
+    // the previous call's hint: the leaf slot of this call's first page, read
+    // while that call's copy was in flight (0: none)
+    uint64_t hsv = 0;
     if constexpr (G::kBlock && kHint) {
-      if (tid == 0 && sc.hint_grid == grid_id() && sc.hint_blk == G::key() && sc.hint_f >= 0) {
-        if (n0 > 0 && sc.hint_fd == fd && sc.hint_page == (off >> shift)) hinted = sc.hint_f;
-        else r64_add_rlx(&c->f_state[sc.hint_f], kRefDec);  // not this call's: drop it
-        sc.hint_f = -1;
+      if (tid == 0 && sc.hint_grid == grid_id() && sc.hint_blk == G::key() && sc.hint_ok) {
+        if (n0 > 0 && sc.hint_fd == fd && sc.hint_page == (off >> shift)) hsv = sc.hint_sv;
+        sc.hint_ok = 0;
       }
     }
     if (n0 > 0) {
@@ -2304,7 +2302,7 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
         const FileSnap fs0 = sc.fs;
         const bool quick_ok =
             q0 == q1 && n0 < (1 << 20) && __isShared(dst) && (((uintptr_t)dst - off) & 15) == 0;
-        if (fast && hinted < 0 && quick_ok && !(c->flags & GFS_F_NO_SPECULATE)) {
+        if (fast && quick_ok && !(c->flags & GFS_F_NO_SPECULATE)) {
           // Speculative one-page hit (lane 0; cnt == 1): a slot whose fill is known
           // complete (no kSlotFill) lets the copy start with the reference still in
           // flight. The reference's old state decides: same generation and no
@@ -2312,8 +2310,10 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
           // the slot read on (a generation is never reused), so the copy is kept;
           // otherwise the reference is dropped, the copy waited out (it may not
           // land after dst is reused) and the call takes the normal path.
-          uint64_t* const sp = leaf_slot(c, fs0, q0, sc.lc_ok ? sc.leaf : nullptr);
-          const uint64_t sv = sp ? ld_rlx64(sp) : 0ull;
+          // (a hinted slot value was read earlier: the same argument holds from
+          // that read on, and a stale one fails the generation check)
+          uint64_t* const sp = hsv ? nullptr : leaf_slot(c, fs0, q0, sc.lc_ok ? sc.leaf : nullptr);
+          const uint64_t sv = hsv ? hsv : sp ? ld_rlx64(sp) : 0ull;
           if ((uint32_t)sv && !((uint32_t)sv & kSlotFill)) {
             const uint32_t fs_ = slot_frame(sv);
             const uint64_t old = a64_add_rlx(&c->f_state[fs_], 1ull);
@@ -2334,7 +2334,7 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
             }
           }
         }
-        int f = quick ? -2 : hinted >= 0 ? hinted : fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
+        int f = quick ? -2 : fast ? lookup_fast(c, fs0, q0 + tid, sc.lc_ok ? sc.leaf : nullptr) : -1;
         if (quick) {
           // the speculative copy is in flight (above)
         } else if (f < 0) {
@@ -2372,13 +2372,16 @@ __device__ inline int64_t gread_t(const gfs_ctx* c, int fd, uint64_t off, uint64
     const uint32_t ph = sc.mbar_phase;
     copy_edges((uint8_t*)dst, frame_ptr(c, (uint32_t)sc.frame[0]) + (off & (P - 1)), (uint32_t)n, tid);
     if constexpr (G::kBlock && kHint) {
-      // hint: look up and reference the next call's first page while the copy flies
+      // hint: read the leaf slot of the next call's first page while the copy
+      // flies (no reference: the next call's speculative copy validates it)
       if (next_off != ~0ull && tid == 0 && fast && next_off < sc.fs.size) {
         sc.hint_grid = grid_id();
         sc.hint_blk = G::key();
         sc.hint_fd = fd;
         sc.hint_page = next_off >> shift;
-        sc.hint_f = lookup_fast(c, sc.fs, sc.hint_page, sc.lc_ok ? sc.leaf : nullptr);
+        uint64_t* const nsp = leaf_slot(c, sc.fs, sc.hint_page, sc.lc_ok ? sc.leaf : nullptr);
+        sc.hint_sv = nsp ? ld_rlx64(nsp) : 0ull;
+        sc.hint_ok = sc.hint_sv != 0;
       }
     }
     mbar_wait(&sc.mbar, ph);
@@ -2409,12 +2412,13 @@ __device__ inline int64_t gread(const gfs_ctx* c, int fd, uint64_t off, uint64_t
 }
 // gread with the offset of the block's NEXT gread on the same file (a split-
 // phase lookup, NEXT-2): while this call's one-page copy into
-// shared memory is in flight, warp 0 looks up and references the page holding
-// next_off, so the next call starts its copy without a lookup. The reference
-// is consumed by the next gread_hint (or dropped by it if the offset differs;
-// next_off = ~0: no further hint) or by gclose of the file. Plain gread does
-// not look at hints (it pays nothing for them), so a block that passed a hint
-// calls gread_hint or gclose next.
+// shared memory is in flight, lane 0 reads the leaf slot of the page holding
+// next_off (no reference is taken), so the next gread_hint starts its
+// speculative copy right after its opening barrier, without a tree access;
+// the copy is validated by the reference as always (a stale slot value fails
+// the generation check and the call takes the normal path). A hint for
+// another offset is ignored; next_off = ~0: no hint. Plain gread does not look
+// at hints (it pays nothing for them).
 __device__ inline int64_t gread_hint(const gfs_ctx* c, int fd, uint64_t off, uint64_t len, void* dst,
                                      uint64_t next_off) {
   return gread_t<detail::BlockGroup, true>(c, fd, off, len, dst, next_off);
