@@ -513,8 +513,9 @@ def hit_phase(X):
                          "note": "1 algorithmic HBM byte per delivered byte (frame read; destination is smem); per GPU"},
             "hint": {"GBps": round(X.ws * gbs(nbytes, X.allmax(mh)), 3), "vs_raw": round(mr / mh, 4),
                      "ms": round(mh, 3), "checksum_eq_oracle": sh == want,
-                     "note": "gread_hint: each call names the block's next offset, whose page is looked up and "
-                             "referenced while the current copy is in flight (split-phase lookup)"},
+                     "note": "gread_hint: each call names the block's next offset, whose leaf slot is read while "
+                             "the current copy is in flight (no reference; the next call's speculative copy "
+                             "starts without a tree access)"},
             "parity": {"checksum_eq_oracle": sg == want, "raw_eq_oracle": sr == want, "hint_eq_oracle": sh == want,
                        "oracle_s": round(oracle_s, 2)},
             "misses_after_warm": st["miss"],
