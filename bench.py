@@ -498,6 +498,17 @@ def hit_phase(X):
         run_l()
         ms_locked = float(np.median(X.timed(run_l, 3)))
         stl = fl.stats()
+    # ablation of the speculative one-page hit copy: the full K4 run with
+    # every hit waiting for its reference before the copy starts
+    with g.GpuFS(cache_bytes=size + (256 << 20), page_size=P, device=X.local, daemon_threads=args.daemon_threads,
+                 timeout_ms=args.timeout_ms, flags=8) as fn:  # 8 = GFS_F_NO_SPECULATE
+        s3, err3 = fn.seqread(path, size, P, grid=296)
+        assert err3 == 0 and s3 == s
+        run_n = lambda: (out.zero_(), fn.randread(path, chunk, d_off, grid, block=args.hit_block,
+                                                  stream=X.stream, sync=False, out=out))
+        X.timed(run_n, 2)
+        tn = X.timed(run_n, reps)
+        sn = int(out[0].item()) & M64
     nbytes = grid * calls * chunk
     mg, sdg = mstd(tg)
     mr, _ = mstd(tr)
@@ -516,7 +527,11 @@ def hit_phase(X):
                      "note": "gread_hint: each call names the block's next offset, whose leaf slot is read while "
                              "the current copy is in flight (no reference; the next call's speculative copy "
                              "starts without a tree access)"},
+            "no_speculate": {"GBps": round(X.ws * gbs(nbytes, X.allmax(mstd(tn)[0])), 3),
+                             "vs_raw": round(mr / mstd(tn)[0], 4), "checksum_eq_oracle": sn == want,
+                             "note": "GFS_F_NO_SPECULATE: one-page hits wait for the reference before the copy"},
             "parity": {"checksum_eq_oracle": sg == want, "raw_eq_oracle": sr == want, "hint_eq_oracle": sh == want,
+                       "no_speculate_eq_oracle": sn == want,
                        "oracle_s": round(oracle_s, 2)},
             "misses_after_warm": st["miss"],
             "k5_locked_ablation": {"calls_per_block": abl_calls, "lockfree_ms": round(ms_lockfree, 3),
@@ -1149,7 +1164,8 @@ def make_summary(line, c2, extra):
     h = extra.get("hit")
     if h:
         s.update({"k4_GBps": h["GBps"], "k4_frac_hbm": h["roofline"]["frac"], "k4_vs_raw": h["vs_raw"],
-                  "k4_parity": h["parity"]["checksum_eq_oracle"]})
+                  "k4_parity": h["parity"]["checksum_eq_oracle"],
+                  "k4_no_speculate_vs_raw": h.get("no_speculate", {}).get("vs_raw")})
     hg = extra.get("hit_global")
     if hg:
         best = max(hg["points"], key=lambda p: p["frac_hbm_2B"])
