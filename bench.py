@@ -692,7 +692,30 @@ def grep_run(X, fs, d, lst, reps, hits, file_ids, chunk=16384, block=128):
                                     chunk=chunk, block=block), 1)
         times += t
     out = fs.grep(d, lst, hits=hits, keep_open=True, stream=X.stream, state=state, chunk=chunk, block=block)
-    return times[0], times[1:], out
+    return times[0], times[1:], out, state
+
+
+def grep_graph_run(X, fs, state, d, lst, reps, hits, chunk=16384, block=128):
+    """The same warm run replayed from a CUDA graph (gfs_grep_graph_create): device ms
+    of each replay and the last replay's output (checked against the oracle by the caller)."""
+    fs.grep_graph(state, d, lst)
+    run = lambda: fs.grep(d, lst, hits=hits, keep_open=True, stream=X.stream, sync=False, state=state, chunk=chunk,
+                          block=block)
+    X.timed(run, 1)
+    X.barrier()
+    t = X.timed(run, reps)
+    out = fs.grep(d, lst, hits=hits, keep_open=True, stream=X.stream, state=state, chunk=chunk, block=block)
+    fs.close_grep_graph(state)
+    return t, out
+
+
+def grep_parity(out, ref, hits):
+    r = {"records": out["records"].tolist() == ref.records.tolist(),
+         "totals": out["totals"].tolist() == ref.totals.tolist(),
+         "digest": tuple(out["digest"]) == tuple(ref.digest), "err": out["summary"]["err"] == 0}
+    if hits:
+        r["hits"] = out["hits"].tolist() == ref.hits.tolist()
+    return r
 
 
 def c1_phase(X):
@@ -702,13 +725,17 @@ def c1_phase(X):
     c = X.shared_input(lambda: gen.c1_corpus(f"{SHM}/gfs_bench_c1", seed=1))
     with g.GpuFS(cache_bytes=1 << 30, page_size=64 << 10, device=X.local, daemon_threads=args.daemon_threads,
                  timeout_ms=args.timeout_ms) as fs:
-        cold, warm, out = grep_run(X, fs, c["dict"], c["list"], args.reps, True, None)
+        cold, warm, out, state = grep_run(X, fs, c["dict"], c["list"], args.reps, True, None)
+        tgr, out_g = grep_graph_run(X, fs, state, c["dict"], c["list"], args.reps, True)
     ref = oracle.grep(c["dict"], c["list"], want_hits=True, nthreads=X.nproc)
     nbytes = ref.bytes
     m, sd = mstd(warm)
+    mg, sdg = mstd(tgr)
     return {"workload": "C1: 64-word dictionary, 16 x 512 KiB synthetic text, 64 KiB pages, cache > corpus",
             "cold_ms": round(cold, 3), "warm_ms": round(m, 3), "warm_ms_std": round(sd, 3),
             "warm_GBps": round(gbs(nbytes, m), 3), "nhits": int(out["digest"][2]),
+            "warm_graph": {"ms": round(mg, 3), "ms_std": round(sdg, 3), "parity": grep_parity(out_g, ref, True),
+                           "note": "the warm run replayed from a CUDA graph (gfs_grep_graph_create)"},
             "parity": {"records": out["records"].tolist() == ref.records.tolist(),
                        "totals": out["totals"].tolist() == ref.totals.tolist(),
                        "digest": tuple(out["digest"]) == tuple(ref.digest),
@@ -731,7 +758,7 @@ def grep_phase(X):
     shard_bytes = int(sum(sizes[i] for i in shard))
     with g.GpuFS(cache_bytes=args.grep_cache_gib << 30, page_size=64 << 10, device=X.local,
                  daemon_threads=args.daemon_threads, max_files=1 << 16, timeout_ms=args.timeout_ms) as fs:
-        cold, warm, out = grep_run(X, fs, c["dict"], lst, args.reps, False, np.asarray(shard, np.uint32))
+        cold, warm, out, _ = grep_run(X, fs, c["dict"], lst, args.reps, False, np.asarray(shard, np.uint32))
         gst = fs.stats()
         # wall clock of one more warm run including the final reduction: NCCL
         # all-reduce of the per-word totals and the digest on the device, the
@@ -758,6 +785,7 @@ def grep_phase(X):
         wall_ms = 1e3 * (time.perf_counter() - t0)
         tot, dig, allrecs = gdist.reduce_grep(X.dist.group.WORLD if X.ws > 1 else None, out["totals"],
                                               out["digest"], out["records"], device=torch.device(X.dev), root=0)
+        tgr, out_g = grep_graph_run(X, fs, state, c["dict"], lst, args.reps, False) if X.ws == 1 else (None, None)
     cold_max = X.allmax(cold)
     m, sd = mstd(warm)
     m_max = X.allmax(m)
@@ -787,6 +815,10 @@ def grep_phase(X):
                          "digest": (ref.digest[0], ref.digest[1]) == (int(dig[0]), int(dig[1]))}
         res["cpu_baseline"] = {"value": round(ref.bytes / dt / 1e9, 4), "unit": "GB/s", "cores": X.nproc,
                                "kind": "oracle", "sample": f"whole C4 corpus ({ref.bytes} B), {X.nproc} threads"}
+        if out_g is not None:
+            mg, sdg = mstd(tgr)
+            res["warm_graph"] = {"ms": round(mg, 3), "ms_std": round(sdg, 3), "parity": grep_parity(out_g, ref, False),
+                                 "note": "the warm run replayed from a CUDA graph (gfs_grep_graph_create)"}
     return res
 
 
@@ -1173,12 +1205,16 @@ def make_summary(line, c2, extra):
                   "hitg_parity": all(p["parity"] for p in hg["points"])})
     c1 = extra.get("c1")
     if c1:
-        s.update({"c1_warm_ms": c1["warm_ms"], "c1_cold_ms": c1["cold_ms"], "c1_parity": all(c1["parity"].values())})
+        s.update({"c1_warm_ms": c1["warm_ms"], "c1_cold_ms": c1["cold_ms"], "c1_parity": all(c1["parity"].values()),
+                  "c1_graph_ms": c1["warm_graph"]["ms"], "c1_graph_parity": all(c1["warm_graph"]["parity"].values())})
     gr = extra.get("grep")
     if gr:
         s.update({"c4_warm_ms": gr["warm"]["ms"], "c4_warm_std": gr["warm"]["ms_std"], "c4_cold_ms": gr["cold"]["ms"],
                   "c4_wall_reduce_ms": gr["wall_with_reduce_ms"], "c4_frac_hbm": gr["roofline_warm"]["frac"],
                   "c4_parity": all(gr.get("parity", {}).values()) if gr.get("parity") else None})
+        if gr.get("warm_graph"):
+            s.update({"c4_graph_ms": gr["warm_graph"]["ms"],
+                      "c4_graph_parity": all(gr["warm_graph"]["parity"].values())})
     mv = extra.get("matvec")
     if mv:
         s.update({"c3_GBps": mv["GBps"], "c3_std": mv["GBps_std"], "c3_link_frac_h2d": mv["roofline"]["frac"],

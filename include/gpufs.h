@@ -315,6 +315,23 @@ int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* lis
              const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
              uint64_t* d_hits, uint64_t* d_summary);
 
+/* The same grep run captured once as a CUDA graph and replayed (the pipeline
+ * is ~16 small kernels: launch-bound for small corpora). gfs_grep_graph_create
+ * captures exactly what gfs_grep would enqueue for these arguments (the path
+ * strings are copied into device memory the graph owns; parameters, buffers and
+ * the cache context are fixed at capture: re-create the graph after gfs_export /
+ * gfs_attach_peer or to change any argument); `stream` is unused (capture runs
+ * on a private stream; nothing executes). gfs_grep_graph_launch enqueues one
+ * run on `stream`: the same results and work-area state as gfs_grep.
+ * Returns 0 or -errno (-EINVAL bad arguments, -ENAMETOOLONG a path,
+ * -EIO capture or instantiation failed). */
+typedef struct gfs_grep_graph gfs_grep_graph;
+int gfs_grep_graph_create(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
+                          const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap,
+                          uint64_t* d_totals, uint64_t* d_hits, uint64_t* d_summary, gfs_grep_graph** out);
+int gfs_grep_graph_launch(gfs_grep_graph* g, void* stream);
+int gfs_grep_graph_destroy(gfs_grep_graph* g);
+
 /* --------------------------------------------------------------------------
  * Out-of-core fp32 matrix-vector product (§5.1.4): y = A x with
  * A a row-major little-endian fp32 file (rows x cols), x a cols-long fp32

@@ -104,6 +104,10 @@ def lib():
             "gfs_run_seqwrite": ([P, P, CS, U64, U64, P, P, P, U32, U32, U32], I),
             "gfs_grep_work_bytes": ([ctypes.POINTER(gfs_grep_params)], U64),
             "gfs_grep": ([P, P, CS, CS, ctypes.POINTER(gfs_grep_params), P, P, U64, P, P, P], I),
+            "gfs_grep_graph_create": ([P, P, CS, CS, ctypes.POINTER(gfs_grep_params), P, P, U64, P, P, P,
+                                       ctypes.POINTER(P)], I),
+            "gfs_grep_graph_launch": ([P, P], I),
+            "gfs_grep_graph_destroy": ([P], I),
             "gfs_matvec": ([P, P, CS, CS, CS, U64, U64, P, P, P, U32, U32], I),
             "gfs_matvec_rows": ([P, P, CS, CS, CS, U64, U64, U64, U64, P, P, P, U32, U32], I),
         }
@@ -255,6 +259,22 @@ def gfs_grep(h, stream, dict_path, list_path, p: gfs_grep_params, d_work, d_rec,
              d_summary):
     return _ck(lib().gfs_grep(h, stream, _b(dict_path), _b(list_path), ctypes.byref(p), d_work, d_rec, rec_cap,
                               d_totals, d_hits, d_summary), "gfs_grep")
+
+
+def gfs_grep_graph_create(h, stream, dict_path, list_path, p: gfs_grep_params, d_work, d_rec, rec_cap, d_totals,
+                          d_hits, d_summary):
+    g = ctypes.c_void_p()
+    _ck(lib().gfs_grep_graph_create(h, stream, _b(dict_path), _b(list_path), ctypes.byref(p), d_work, d_rec,
+                                    rec_cap, d_totals, d_hits, d_summary, ctypes.byref(g)), "gfs_grep_graph_create")
+    return g
+
+
+def gfs_grep_graph_launch(g, stream):
+    return _ck(lib().gfs_grep_graph_launch(g, stream), "gfs_grep_graph_launch")
+
+
+def gfs_grep_graph_destroy(g):
+    return _ck(lib().gfs_grep_graph_destroy(g), "gfs_grep_graph_destroy")
 
 
 def gfs_matvec(h, stream, a_path, x_path, y_path, rows, cols, d_x, d_y, d_err, grid, block):

@@ -283,15 +283,18 @@ class GpuFS:
 
         Capacities come from file metadata (stat), never from file contents: the
         contents are read on the GPU through gopen/gread."""
-        from . import GREP_SUMMARY, gfs_grep
+        from . import GREP_SUMMARY, gfs_grep, gfs_grep_graph_launch
         if state is None:
             state = self.grep_state(dict_path, list_path, hits, chunk, grid, block, keep_open, pair_cap, hit_cap,
                                     corpus_cap, rec_cap, file_ids, whole_max, scan)
         p = state["p"]
         s, sp = self._stream(stream)
-        gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
-                 state["rec_cap"], state["totals"].data_ptr(),
-                 state["hits"].data_ptr() if state["hits"] is not None else None, state["summary"].data_ptr())
+        if state.get("graph") is not None:  # the run captured by grep_graph (same arguments)
+            gfs_grep_graph_launch(state["graph"], sp)
+        else:
+            gfs_grep(self.h, sp, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
+                     state["rec_cap"], state["totals"].data_ptr(),
+                     state["hits"].data_ptr() if state["hits"] is not None else None, state["summary"].data_ptr())
         if not sync:
             return state
         s.synchronize()
@@ -316,6 +319,24 @@ class GpuFS:
             out["hits"] = hh[order]
         out["state"] = state
         return out
+
+    def grep_graph(self, state, dict_path, list_path):
+        """Capture one grep run with these arguments as a CUDA graph (gfs_grep_graph_create);
+        grep(state=state, ...) then replays it (one graph launch instead of ~16 kernel
+        launches). Returns the state; close_grep_graph(state) frees the graph."""
+        from . import gfs_grep_graph_create
+        p = state["p"]
+        state["graph"] = gfs_grep_graph_create(
+            self.h, None, dict_path, list_path, p, state["work"].data_ptr(), state["rec"].data_ptr(),
+            state["rec_cap"], state["totals"].data_ptr(),
+            state["hits"].data_ptr() if state["hits"] is not None else None, state["summary"].data_ptr())
+        return state
+
+    @staticmethod
+    def close_grep_graph(state):
+        from . import gfs_grep_graph_destroy
+        if state.get("graph") is not None:
+            gfs_grep_graph_destroy(state.pop("graph"))
 
     # mat-vec -------------------------------------------------------------------
     def matvec(self, a_path, x_path, y_path, rows, cols, grid=None, block=256, stream=None, sync=True, state=None,

@@ -1684,24 +1684,33 @@ uint32_t wscan_slots() {
   return v;
 }
 
-}  // namespace
-
-GFS_API uint64_t gfs_grep_work_bytes(const gfs_grep_params* p) { return p ? layout(p).total : 0; }
-
-GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
-                     const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
-                     uint64_t* d_hits, uint64_t* d_summary) {
-  if (!h || !dict_path || !list_path || !p || !d_work || !d_totals || !d_summary || p->max_files == 0 ||
-      p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 || (p->chunk & 15) ||
-      p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31) || p->scan > 1)
-    return -EINVAL;
+bool grep_params_ok(const gfs_grep_params* p) {
+  if (!p || p->max_files == 0 || p->max_words == 0 || p->max_words >= (1u << 26) || p->chunk == 0 ||
+      (p->chunk & 15) || p->grid == 0 || p->block == 0 || p->block > 256 || (p->block & 31) || p->scan > 1)
+    return false;
   const bool wscan = p->scan == 1;
-  if (!wscan && p->chunk + kPre + kHalo > 65536) return -EINVAL;  // 16-bit token offsets into the item buffer
+  if (!wscan && p->chunk + kPre + kHalo > 65536) return false;  // 16-bit token offsets into the item buffer
   // warp scan: 1 KiB steps never straddle a chunk; an item has < 2^16 tokens
   // and a word index fits the 16-bit key of a count slot
   if (wscan && ((p->chunk & (kWStep - 1)) || p->chunk > 65536 || p->whole_max > 65536 || p->max_words >= 65535))
-    return -EINVAL;
-  cudaStream_t s = (cudaStream_t)stream;
+    return false;
+  return true;
+}
+
+std::string list_dir(const char* list_path) {
+  const char* slash = strrchr(list_path, '/');
+  std::string dir = slash ? std::string(list_path, (size_t)(slash - list_path)) : std::string(".");
+  if (dir.empty()) dir = "/";  // a list at the root: "/" + "/" + line still resolves
+  return dir;
+}
+
+// Everything one grep run enqueues on stream s, given the staged path strings
+// (device memory) and the validated parameters: shared by gfs_grep and the
+// CUDA-graph path (gfs_grep_graph), which captures exactly this sequence.
+int grep_enqueue(gfs_handle* h, cudaStream_t s, const char* d_dict, const char* d_list, const char* d_dir,
+                 uint32_t dir_len, const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap,
+                 uint64_t* d_totals, uint64_t* d_hits, uint64_t* d_summary, unsigned long long* prof) {
+  const bool wscan = p->scan == 1;
   const Layout L = layout(p);
   uint8_t* base = (uint8_t*)d_work;
   GrepWork w;
@@ -1744,28 +1753,8 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   w.filt = (uint32_t*)(base + L.off[16]);
   w.filt_log2 = L.flog2;
 
-  // path arguments: dictionary, list, the list's directory (relative lines)
-  gfs_launch::ArgStage as(h, s);
-  std::string dir;
-  {
-    const char* slash = strrchr(list_path, '/');
-    dir = slash ? std::string(list_path, (size_t)(slash - list_path)) : std::string(".");
-    if (dir.empty()) dir = "/";  // a list at the root: "/" + "/" + line still resolves
-  }
-  const char* strs[3] = {dict_path, list_path, dir.c_str()};
-  if (const int e = as.stage(strs, 3)) return e;
-  const char* d_dict = as.str(0);
-  const char* d_list = as.str(1);
-  const char* d_dir = as.str(2);
-
   const gfs_ctx c = gfs_launch::ctx_val(h);
-  static unsigned long long* d_prof = nullptr;  // GFS_GREP_PROF=1 (diagnostics only)
-  w.prof = nullptr;
-  if (getenv("GFS_GREP_PROF") && *getenv("GFS_GREP_PROF") == '1') {
-    if (!d_prof && cudaMalloc((void**)&d_prof, 8 * sizeof(unsigned long long)) != cudaSuccess) d_prof = nullptr;
-    if (d_prof) cudaMemsetAsync(d_prof, 0, 8 * sizeof(unsigned long long), s);
-    w.prof = d_prof;
-  }
+  w.prof = prof;
   const uint32_t smem = wscan ? (p->block / 32) * WarpSmemLayout::bytes(w.cslots) : scan_smem(p->chunk, p->block, w.cslots);
   if (smem > 200 * 1024) return -EINVAL;
   if (wscan) cudaFuncSetAttribute(k_grep_wscan, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -1788,7 +1777,7 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   k_grep_list_emit<<<list_blocks, 256, 0, s>>>(w, p->max_files);
   // gopen is collective with one leader thread: many one-warp blocks keep
   // more opens in flight (host RPCs when cold, L2 round trips when warm)
-  k_grep_open<<<nsm * 16, 32, 0, s>>>(c, w, d_dir, (uint32_t)dir.size(), p->max_files);
+  k_grep_open<<<nsm * 16, 32, 0, s>>>(c, w, d_dir, dir_len, p->max_files);
   k_grep_items<<<nsm * 2, 256, 0, s>>>(w);
   cudaMemsetAsync(d_totals, 0, (size_t)p->max_words * 8, s);
   // persistent scan grid: every resident block slot once (p->grid caps it)
@@ -1810,9 +1799,40 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   }
   k_grep_hold<<<1, 32, 0, s>>>(c, d_dict, d_list, w, 1, (int)p->keep_open);
   k_grep_summary<<<1, 32, 0, s>>>(w, d_summary);
-  if (w.prof) {
+  return 0;
+}
+
+}  // namespace
+
+GFS_API uint64_t gfs_grep_work_bytes(const gfs_grep_params* p) { return p ? layout(p).total : 0; }
+
+GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
+                     const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap, uint64_t* d_totals,
+                     uint64_t* d_hits, uint64_t* d_summary) {
+  if (!h || !dict_path || !list_path || !d_work || !d_totals || !d_summary || !grep_params_ok(p)) return -EINVAL;
+  cudaStream_t s = (cudaStream_t)stream;
+  // path arguments: dictionary, list, the list's directory (relative lines)
+  gfs_launch::ArgStage as(h, s);
+  const std::string dir = list_dir(list_path);
+  const char* strs[3] = {dict_path, list_path, dir.c_str()};
+  if (const int e = as.stage(strs, 3)) return e;
+  const char* d_dict = as.str(0);
+  const char* d_list = as.str(1);
+  const char* d_dir = as.str(2);
+
+  static unsigned long long* d_prof = nullptr;  // GFS_GREP_PROF=1 (diagnostics only)
+  unsigned long long* prof = nullptr;
+  if (getenv("GFS_GREP_PROF") && *getenv("GFS_GREP_PROF") == '1') {
+    if (!d_prof && cudaMalloc((void**)&d_prof, 8 * sizeof(unsigned long long)) != cudaSuccess) d_prof = nullptr;
+    if (d_prof) cudaMemsetAsync(d_prof, 0, 8 * sizeof(unsigned long long), s);
+    prof = d_prof;
+  }
+  if (const int e = grep_enqueue(h, s, d_dict, d_list, d_dir, (uint32_t)dir.size(), p, d_work, d_rec, rec_cap,
+                                 d_totals, d_hits, d_summary, prof))
+    return e;
+  if (prof) {
     unsigned long long pv[8];
-    cudaMemcpyAsync(pv, w.prof, sizeof(pv), cudaMemcpyDeviceToHost, s);
+    cudaMemcpyAsync(pv, prof, sizeof(pv), cudaMemcpyDeviceToHost, s);
     cudaStreamSynchronize(s);
     double tot = 0;
     for (int i = 0; i < 7; ++i) tot += (double)pv[i];
@@ -1825,4 +1845,81 @@ GFS_API int gfs_grep(gfs_handle* h, void* stream, const char* dict_path, const c
   const cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) fprintf(stderr, "gfs_grep: launch failed: %s\n", cudaGetErrorString(e));
   return e == cudaSuccess ? 0 : -EIO;
+}
+
+// ------------------------------------------------------------------ CUDA graph
+// A grep run captured once as a CUDA graph and replayed: the pipeline is ~16
+// small kernels, launch-bound for small corpora (C1). The path strings live in
+// device memory the graph owns (not in the per-call argument slots), the
+// parameters and the cache context are fixed at capture: re-create the graph
+// after gfs_export / gfs_attach_peer or to change any argument.
+struct gfs_grep_graph {
+  cudaGraphExec_t exec = nullptr;
+  char* d_str = nullptr;
+  int device = 0;
+};
+
+GFS_API int gfs_grep_graph_create(gfs_handle* h, void* stream, const char* dict_path, const char* list_path,
+                                  const gfs_grep_params* p, void* d_work, uint32_t* d_rec, uint64_t rec_cap,
+                                  uint64_t* d_totals, uint64_t* d_hits, uint64_t* d_summary, gfs_grep_graph** out) {
+  if (!h || !dict_path || !list_path || !d_work || !d_totals || !d_summary || !out || !grep_params_ok(p))
+    return -EINVAL;
+  const std::string dir = list_dir(list_path);
+  const char* strs[3] = {dict_path, list_path, dir.c_str()};
+  for (const char* x : strs)
+    if (strlen(x) >= GFS_MAX_PATH) return -ENAMETOOLONG;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  auto* g = new gfs_grep_graph();
+  g->device = gfs_internal_device(h);
+  cudaSetDevice(g->device);
+  char hs[3 * GFS_MAX_PATH] = {};
+  for (int i = 0; i < 3; ++i) memcpy(hs + i * GFS_MAX_PATH, strs[i], strlen(strs[i]) + 1);
+  cudaStream_t cs = nullptr;
+  cudaGraph_t graph = nullptr;
+  int rc = -EIO;
+  if (cudaMalloc((void**)&g->d_str, sizeof(hs)) == cudaSuccess &&
+      cudaMemcpy(g->d_str, hs, sizeof(hs), cudaMemcpyHostToDevice) == cudaSuccess &&
+      cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking) == cudaSuccess &&
+      cudaStreamBeginCapture(cs, cudaStreamCaptureModeRelaxed) == cudaSuccess) {
+    const int e = grep_enqueue(h, cs, g->d_str, g->d_str + GFS_MAX_PATH, g->d_str + 2 * GFS_MAX_PATH,
+                               (uint32_t)dir.size(), p, d_work, d_rec, rec_cap, d_totals, d_hits, d_summary, nullptr);
+    const cudaError_t ec = cudaStreamEndCapture(cs, &graph);
+    if (e) rc = e;
+    else if (ec == cudaSuccess && graph && cudaGraphInstantiate(&g->exec, graph, 0) == cudaSuccess) rc = 0;
+  }
+  if (graph) cudaGraphDestroy(graph);
+  if (cs) cudaStreamDestroy(cs);
+  (void)cudaGetLastError();
+  (void)stream;
+  cudaSetDevice(prev);
+  if (rc) {
+    if (g->d_str) cudaFree(g->d_str);
+    delete g;
+    return rc;
+  }
+  *out = g;
+  return 0;
+}
+
+GFS_API int gfs_grep_graph_launch(gfs_grep_graph* g, void* stream) {
+  if (!g || !g->exec) return -EINVAL;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(g->device);
+  const cudaError_t e = cudaGraphLaunch(g->exec, (cudaStream_t)stream);
+  cudaSetDevice(prev);
+  return e == cudaSuccess ? 0 : -EIO;
+}
+
+GFS_API int gfs_grep_graph_destroy(gfs_grep_graph* g) {
+  if (!g) return -EINVAL;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(g->device);
+  if (g->exec) cudaGraphExecDestroy(g->exec);
+  if (g->d_str) cudaFree(g->d_str);
+  cudaSetDevice(prev);
+  delete g;
+  return 0;
 }

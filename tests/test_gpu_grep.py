@@ -187,3 +187,25 @@ def test_whole_file_count_table_spill(g, shmdir):
         out = fs.grep(os.path.join(shmdir, "d.bin"), os.path.join(shmdir, "l.txt"), hits=True, chunk=4096,
                       whole_max=31 * 4096, grid=4)
     compare(out, ref)
+
+
+def test_grep_cuda_graph_replays(g, shmdir):
+    """The grep run captured as a CUDA graph (gfs_grep_graph_create) and replayed:
+    every replay equals the oracle (records, totals, digest, the full hit list on C1;
+    a C4-shape corpus with files kept open across replays), like direct calls."""
+    c = gen.c1_corpus(os.path.join(shmdir, "c1g"), seed=5)
+    ref = oracle.grep(c["dict"], c["list"], nthreads=4)
+    c4 = gen.c4_corpus(os.path.join(shmdir, "c4g"), seed=16, nfiles=300, total_bytes=6 << 20, nwords=2000)
+    ref4 = oracle.grep(c4["dict"], c4["list"], want_hits=False)
+    with g.GpuFS(cache_bytes=1 << 30, page_size=64 << 10, timeout_ms=30000, daemon_threads=4, max_files=1024) as fs:
+        st = fs.grep_state(c["dict"], c["list"], hits=True)
+        fs.grep_graph(st, c["dict"], c["list"])
+        for _ in range(3):
+            compare(fs.grep(c["dict"], c["list"], hits=True, state=st), ref)
+        fs.close_grep_graph(st)
+        st4 = fs.grep_state(c4["dict"], c4["list"], keep_open=True, chunk=4096)
+        compare(fs.grep(c4["dict"], c4["list"], keep_open=True, chunk=4096, state=st4), ref4, hits=False)
+        fs.grep_graph(st4, c4["dict"], c4["list"])
+        for _ in range(3):
+            compare(fs.grep(c4["dict"], c4["list"], keep_open=True, chunk=4096, state=st4), ref4, hits=False)
+        fs.close_grep_graph(st4)
