@@ -14,7 +14,10 @@ extern "C" int gfs_internal_device(gfs_handle* h);
 // The host copy of the handle's context (what gfs_device_ctx points to on the
 // device, kept in step with it): launchers pass it BY VALUE as a
 // __grid_constant__ kernel parameter, so the kernel reads the context's
-// fields from the constant bank instead of L1/L2.
+// fields from the constant bank instead of L1/L2. Launchers copy it without a
+// lock: gfs_export / gfs_attach_peer (the only calls that change it after
+// gfs_init) must not run concurrently with launches on the same handle from
+// other threads (as before, when kernels read the device copy they update).
 extern "C" const gfs_ctx* gfs_internal_host_ctx(gfs_handle* h);
 
 namespace gfs_launch {
