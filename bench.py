@@ -1270,7 +1270,7 @@ def main():
     ap.add_argument("--fig4-reps", type=int, default=3)
     ap.add_argument("--c5-mib", type=int, default=512)
     ap.add_argument("--c5-iters", type=int, default=3)
-    ap.add_argument("--c5-sync-grid", type=int, default=8)
+    ap.add_argument("--c5-sync-grid", type=int, default=128)  # gfsync blocks (8: 25, 32: 28, 128: 30 GB/s)
     ap.add_argument("--mv-rows", type=int, default=11200)  # 5.6 GB (Fig. 8's 5600 MB point x2)
     ap.add_argument("--mv-passes", type=int, default=3)
     ap.add_argument("--grep-files", type=int, default=30000)
