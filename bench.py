@@ -1253,7 +1253,7 @@ def main():
                                                             # (tools/k4_occ.py: 96 x 10 measured best)
     ap.add_argument("--hit-calls", type=int, default=820)  # ~1.21 M calls in all (1184 x 1024 before)
     ap.add_argument("--hg-gib", type=int, default=16, help="hit->global file size (GiB)")
-    ap.add_argument("--hg-grid", type=int, default=592)
+    ap.add_argument("--hg-grid", type=int, default=2368)  # 592: 0.850, 1184: 0.866, 2368: 0.885 of HBM (2 MiB)
     ap.add_argument("--ref-sample-mib", type=int, default=2048)
     ap.add_argument("--timeout-ms", type=int, default=60000)
     ap.add_argument("--no-hit", action="store_true")
