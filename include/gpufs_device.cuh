@@ -2852,6 +2852,11 @@ __device__ inline void* gmmap_t(const gfs_ctx* c, void* addr, uint64_t len, int 
     }
     G::sync();
   }
+  if constexpr (G::kBlock) {  // NEXT-2: read-ahead of a sequential mapper of a read-only file (warp 0)
+    if (c->readahead && sc.ret == 1 && sc.aux > 0 && tid < 32 && !(sc.fs.oflags & GFS_O_WRITABLE) && !c->npeers &&
+        ld_rlx64(&c->files[sc.fs.fdx].zc) == 0)
+      ra_after<G>(c, sc, sc.fs, fd, off, (uint64_t)sc.aux);
+  }
   if (mapped_len) *mapped_len = sc.aux > 0 ? (uint64_t)sc.aux : 0;
   if (err_out) *err_out = sc.aux < 0 ? (int)sc.aux : 0;
   void* const r = sc.ptr;

@@ -158,3 +158,22 @@ def test_frames_fewer_than_held_pages_enomem(g, shmdir):
         assert fs.stats()["enomem"] > 0
         ret, dst, dstoff = fs.gread_calls(path, np.array([P], np.uint64), np.array([2 * P], np.uint64), grid=1)
         assert int(ret[0]) == 2 * P and dst[:2 * P].tobytes() == oracle.pread(path, size, P, 2 * P)
+
+
+@pytest.mark.parametrize("P,cache_pages,ra,grid", [(65536, 4096, 4, 4), (65536, 48, 8, 8), (1 << 21, 12, 2, 3)])
+def test_readahead_gmmap_sweep_bytes(g, shmdir, P, cache_pages, ra, grid):
+    """Read-ahead behind a sequential gmmap mapper (K1 shape, NEXT-2): the same checksum
+    as the oracle with the next pages fetched ahead, in a cache larger and smaller than
+    the file; read-ahead fills are posted and adopted or reaped, nothing times out."""
+    size = 40 * (1 << 20) + 4321 if P >= (1 << 21) else 300 * P + 999
+    path = gen.splitmix_file(os.path.join(shmdir, "ram.bin"), size, seed=37)
+    total = size - (size % 8)
+    want = oracle.checksum(path, 0, total)
+    with _fs(g, cache_bytes=cache_pages * P, page_size=P, readahead=ra, max_batch=4) as fs:
+        for rep in range(3):
+            s, err = fs.seqread(path, total, P, grid=grid, use_mmap=True)
+            assert err == 0 and s == want, rep
+        st = fs.stats()
+        assert st["ra_issued"] > 0
+        assert st["ra_adopted"] + st["ra_reaped"] <= st["ra_issued"]
+        assert st["timeout"] == 0 and st["enomem"] == 0
